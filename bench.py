@@ -1,0 +1,349 @@
+#!/usr/bin/env python
+"""Benchmark: HD->SD fused ArrayOL downscale, frames/s and achieved HBM GB/s.
+
+Contract (driver): `python bench.py --gpus N --steps K --warmup W [--impl reference]`,
+launched under torchrun for N > 1 (one process per GPU, NCCL).  Rank 0 prints
+ONE JSON line.
+
+Workload (BASELINE.json configs[1]): a 300-frame 1920x1080 3-channel synthetic
+int32 stream per GPU (weak scaling: each rank owns its own 300 frames, global
+frame indices rank*300 .. rank*300+299).  One step = one aol_downscale_frame
+call over the whole 300-frame batch, checksum epilogue included: every row of
+SURVEY.md 8(a) (a1-a9) runs inside the step.  Inputs (7.46 GB) are larger than
+the 126 MB L2, so no explicit flush is needed between steps.
+
+`value` is device-timed (CUDA events on the launching stream, barrier + sync on
+both sides, max over ranks); `e2e` is the same metric through the host-buffer
+C-ABI call (aol_downscale_frame_host: pinned H2D, kernel, D2H inside the timed
+region).  `cpu_baseline` times the CPU oracle (oracle/, test infrastructure)
+on a bounded sample of the same workload -- a reported baseline, not a target.
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import statistics
+import sys
+import threading
+import time
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+if ROOT not in sys.path:
+    sys.path.insert(0, ROOT)
+
+METRIC = "HD->SD downscale frames/sec (1/2/4/8 B200) and achieved HBM GB/s vs peak"
+FALLBACK_HBM_GBS = 6650.0  # /opt/skills/guides/B200_PROFILING.md fallback
+
+
+def parse():
+    p = argparse.ArgumentParser()
+    p.add_argument("--gpus", type=int, default=1)
+    p.add_argument("--steps", type=int, default=100)
+    p.add_argument("--warmup", type=int, default=5)
+    p.add_argument("--impl", choices=["aol", "reference"], default="aol")
+    p.add_argument("--frames", type=int, default=300, help="frames per GPU (configs[1]: 300)")
+    p.add_argument("--channels", type=int, default=3)
+    p.add_argument("--H", type=int, default=1080)
+    p.add_argument("--W", type=int, default=1920)
+    p.add_argument("--seed", type=int, default=0)
+    p.add_argument("--dtype", choices=["i32", "u8"], default="i32")
+    p.add_argument("--opts", type=str, default="", help='launch options JSON, e.g. {"ctas_per_sm":2}')
+    p.add_argument("--e2e-steps", type=int, default=3)
+    p.add_argument("--no-e2e", action="store_true")
+    p.add_argument("--no-cpu-baseline", action="store_true")
+    return p.parse_args()
+
+
+def workload_name(a):
+    return f"{a.frames}-frame {a.W}x{a.H} {a.channels}-channel synthetic stream per GPU, fused h+v downscale"
+
+
+def bytes_per_frame(a):
+    es = 4 if a.dtype == "i32" else 1
+    Ho, Wo = 4 * (a.H // 9), 3 * (a.W // 8)
+    return a.channels * (a.H * a.W * es + Ho * Wo * 4)
+
+
+def measured_peak():
+    path = os.path.join(ROOT, "MEASURED_PEAKS.json")
+    try:
+        with open(path) as f:
+            d = json.load(f)
+        return float(d["hbm_gbs"]), "measured (MEASURED_PEAKS.json hbm_gbs, copy read+write)"
+    except Exception:
+        return FALLBACK_HBM_GBS, "fallback (B200_PROFILING.md)"
+
+
+def ncu_traffic(a):
+    """Per-launch DRAM bytes from the committed `ncu --set full` summary, if it matches this workload."""
+    path = os.path.join(ROOT, "profiles", "ncu_traffic.json")
+    try:
+        with open(path) as f:
+            d = json.load(f)
+        key = f"{a.frames}x{a.channels}x{a.H}x{a.W}:{a.dtype}"
+        e = d.get(key)
+        return None if e is None else float(e["dram_bytes_per_launch"])
+    except Exception:
+        return None
+
+
+class ClockSampler:
+    """Samples SM clocks and throttle reasons with NVML during the timed region."""
+
+    def __init__(self, device_index):
+        self.samples, self.reasons, self.max_mhz = [], set(), None
+        self._stop = threading.Event()
+        self._ok = False
+        try:
+            import pynvml
+
+            pynvml.nvmlInit()
+            self._nv = pynvml
+            self._h = pynvml.nvmlDeviceGetHandleByIndex(device_index)
+            self.max_mhz = pynvml.nvmlDeviceGetMaxClockInfo(self._h, pynvml.NVML_CLOCK_SM)
+            self._ok = True
+        except Exception:
+            pass
+        self._names = {}
+        if self._ok:
+            nv = self._nv
+            for name in ("HwSlowdown", "HwThermalSlowdown", "SwThermalSlowdown", "SwPowerCap", "HwPowerBrakeSlowdown",
+                         "SyncBoost", "ApplicationsClocksSetting", "DisplayClockSetting"):
+                attr = "nvmlClocksThrottleReason" + name
+                if hasattr(nv, attr):
+                    self._names[getattr(nv, attr)] = {
+                        "HwSlowdown": "hw_slowdown", "HwThermalSlowdown": "hw_thermal_slowdown",
+                        "SwThermalSlowdown": "sw_thermal_slowdown", "SwPowerCap": "sw_power_cap",
+                        "HwPowerBrakeSlowdown": "hw_power_brake_slowdown", "SyncBoost": "sync_boost",
+                        "ApplicationsClocksSetting": "applications_clocks_setting",
+                        "DisplayClockSetting": "display_clock_setting"}[name]
+
+    def _run(self):
+        nv = self._nv
+        while not self._stop.is_set():
+            try:
+                self.samples.append(nv.nvmlDeviceGetClockInfo(self._h, nv.NVML_CLOCK_SM))
+                mask = nv.nvmlDeviceGetCurrentClocksThrottleReasons(self._h)
+                for bit, name in self._names.items():
+                    if mask & bit:
+                        self.reasons.add(name)
+            except Exception:
+                pass
+            time.sleep(0.005)
+
+    def __enter__(self):
+        if self._ok:
+            self._t = threading.Thread(target=self._run, daemon=True)
+            self._t.start()
+        return self
+
+    def __exit__(self, *exc):
+        if self._ok:
+            self._stop.set()
+            self._t.join()
+
+    def summary(self):
+        if not self._ok:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": ["nvml_unavailable"]}
+        return {"sm_mhz": statistics.median(self.samples) if self.samples else None, "sm_max_mhz": self.max_mhz,
+                "reasons": sorted(self.reasons), "samples": len(self.samples)}
+
+
+def cpu_baseline(a, gpu_cs=None, frame0=0, steps=1):
+    """Time the CPU oracle (as it stands, OpenMP across planes) on a bounded sample.
+    Returns (frames_per_s, info).  Also checks oracle checksums against the GPU's for
+    the unique sample frames when gpu_cs is given."""
+    import numpy as np
+
+    import oracle
+    import synth
+
+    cores = os.cpu_count() or 1
+    nthreads = max(1, min(cores, oracle.max_threads() if oracle.max_threads() > 0 else cores))
+    sample = max(8, min(a.frames, 2 * nthreads))
+    uniq = min(sample, 8)
+    xu = synth.frames(a.seed, frame0, uniq, a.channels, a.H, a.W, "uniform")
+    if a.dtype == "u8":
+        xu = xu.astype(np.int32)
+    reps = (sample + uniq - 1) // uniq
+    x = np.ascontiguousarray(np.concatenate([xu] * reps)[:sample])
+    oracle.downscale_frame(x[:1], nthreads=1)  # warm the library
+    times = []
+    cs = None
+    for _ in range(steps):
+        t0 = time.perf_counter()
+        _, cs = oracle.downscale_frame(x, nthreads=nthreads)
+        times.append(time.perf_counter() - t0)
+    dt = statistics.median(times)
+    info = {"cores": nthreads, "sample": f"{sample} frames of the workload ({uniq} unique, seed {a.seed}, "
+                                        f"frames {frame0}..{frame0 + uniq - 1} repeated), OpenMP over planes, "
+                                        f"median of {steps}", "seconds": dt}
+    if gpu_cs is not None:
+        info["parity_sample_ok"] = bool(np.array_equal(cs[:uniq], gpu_cs[:uniq]))
+    return sample / dt, info
+
+
+def run_reference(a, rank):
+    """--impl reference: the CPU oracle is this tier's reference arm (rank 0 only)."""
+    if rank != 0:
+        return
+    steps, warm = a.steps, a.warmup
+    import oracle  # noqa: F401
+
+    fps_list = []
+    # warm-up + timed steps; each step is a bounded sample of the workload
+    for i in range(warm + steps):
+        fps, info = cpu_baseline(a, steps=1)
+        if i >= warm:
+            fps_list.append(fps)
+    value = statistics.median(fps_list)
+    line = {
+        "metric": METRIC, "value": value, "unit": "frames/s", "n_gpus": a.gpus, "steps": steps, "warmup": warm,
+        "ms_per_step": 1000.0 * info["seconds"], "higher_is_better": True, "scaling": "weak",
+        "vs_baseline": None, "dtype": a.dtype, "data": "synthetic",
+        "config": {"workload": workload_name(a), "frames": a.frames, "H": a.H, "W": a.W,
+                   "channels": a.channels, "l2": "inputs larger than L2 (no flush)"},
+        "impl": "reference",
+        "cpu_baseline": {"value": value, "unit": "frames/s", "cores": info["cores"], "kind": "oracle",
+                         "sample": info["sample"]},
+        "e2e": {"value": value, "unit": "frames/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
+    }
+    print(json.dumps(line), flush=True)
+
+
+def main():
+    a = parse()
+    rank = int(os.environ.get("RANK", "0"))
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    local_rank = int(os.environ.get("LOCAL_RANK", "0"))
+
+    if a.impl == "reference":
+        run_reference(a, rank)
+        return
+
+    import numpy as np
+    import torch
+    import torch.distributed as dist
+
+    import paper_conf_ipps_guortgbs11_b200 as aol
+
+    torch.cuda.set_device(local_rank)
+    dev = torch.device("cuda", local_rank)
+    if world > 1:
+        dist.init_process_group("nccl", device_id=dev)
+    opts = json.loads(a.opts) if a.opts else None
+
+    F, C, H, W = a.frames, a.channels, a.H, a.W
+    frame0 = rank * F
+    tdtype = torch.int32 if a.dtype == "i32" else torch.uint8
+    x = aol.synth_frames(a.seed, frame0, F, C, H, W, "uniform", dtype=tdtype, device=dev)
+    z = torch.empty((F, C, 4 * (H // 9), 3 * (W // 8)), dtype=torch.int32, device=dev)
+    cs = torch.empty(F, dtype=torch.uint64, device=dev)
+    plan = aol.downscale_frame_plan(F, C, H, W, dtype=tdtype, opts=opts)
+    stream = torch.cuda.current_stream(dev)
+
+    for _ in range(a.warmup):
+        aol.downscale_frame(x, out=z, checksums=cs, opts=opts)
+    torch.cuda.synchronize(dev)
+
+    starts = [torch.cuda.Event(enable_timing=True) for _ in range(a.steps)]
+    ends = [torch.cuda.Event(enable_timing=True) for _ in range(a.steps)]
+    t_begin = torch.cuda.Event(enable_timing=True)
+    t_end = torch.cuda.Event(enable_timing=True)
+    if world > 1:
+        dist.barrier()
+    torch.cuda.synchronize(dev)
+    with ClockSampler(local_rank) as clk:
+        t_begin.record(stream)
+        for i in range(a.steps):
+            starts[i].record(stream)
+            aol.downscale_frame(x, out=z, checksums=cs, opts=opts)
+            ends[i].record(stream)
+        t_end.record(stream)
+        torch.cuda.synchronize(dev)
+    if world > 1:
+        dist.barrier()
+    elapsed_ms = t_begin.elapsed_time(t_end)
+    launch_ms = [s.elapsed_time(e) for s, e in zip(starts, ends)]
+
+    # max over ranks (NCCL), and gather per-rank checksums + timings (the only cross-GPU traffic)
+    t = torch.tensor([elapsed_ms], dtype=torch.float64, device=dev)
+    cs_all = None
+    if world > 1:
+        dist.all_reduce(t, op=dist.ReduceOp.MAX)
+        gathered = torch.empty(world * F, dtype=torch.int64, device=dev)
+        dist.all_gather_into_tensor(gathered, cs.view(torch.int64))
+        cs_all = gathered.cpu().numpy().view(np.uint64)
+    max_ms = float(t.item())
+
+    # e2e through the host-buffer C-ABI call
+    e2e = None
+    if not a.no_e2e:
+        x_host = torch.empty(x.shape, dtype=x.dtype, pin_memory=True)
+        x_host.copy_(x)
+        z_host = torch.empty(z.shape, dtype=torch.int32, pin_memory=True)
+        chunk = 20
+        ws = torch.empty(aol.host_workspace_bytes(chunk, C, H, W, tdtype), dtype=torch.uint8, device=dev)
+        streams = [torch.cuda.Stream(device=dev) for _ in range(3)]
+        aol.downscale_frame_host(x_host, out=z_host, chunk_frames=chunk, workspace=ws, streams=streams, device=dev)
+        if world > 1:
+            dist.barrier()
+        t0 = time.perf_counter()
+        for _ in range(a.e2e_steps):
+            _, cs_h = aol.downscale_frame_host(x_host, out=z_host, chunk_frames=chunk, workspace=ws,
+                                               streams=streams, device=dev)
+        e2e_s = time.perf_counter() - t0
+        te = torch.tensor([e2e_s], dtype=torch.float64, device=dev)
+        if world > 1:
+            dist.all_reduce(te, op=dist.ReduceOp.MAX)
+        e2e_s = float(te.item())
+        same = bool(torch.equal(cs_h.view(torch.int64), cs.cpu().view(torch.int64)))
+        e2e = {"value": world * F * a.e2e_steps / e2e_s, "unit": "frames/s",
+               "h2d_bytes_per_step": int(x.numel() * x.element_size()),
+               "d2h_bytes_per_step": int(z.numel() * 4 + F * 8), "steps": a.e2e_steps,
+               "chunk_frames": chunk, "checksums_match_device_path": same,
+               "timing": "host wall clock around the blocking call, max over ranks"}
+
+    if rank != 0:
+        if world > 1:
+            dist.destroy_process_group()
+        return
+
+    value = world * F * a.steps / (max_ms / 1000.0)
+    bpf = bytes_per_frame(a)
+    avg_launch_s = statistics.mean(launch_ms) / 1000.0
+    achieved = bpf * F / avg_launch_s / 1e9
+    peak, peak_src = measured_peak()
+    traffic = ncu_traffic(a)
+    line = {
+        "metric": METRIC, "value": value, "unit": "frames/s", "n_gpus": world, "steps": a.steps,
+        "warmup": a.warmup, "ms_per_step": max_ms / a.steps, "higher_is_better": True, "scaling": "weak",
+        "vs_baseline": None, "dtype": a.dtype, "data": "synthetic",
+        "config": {"workload": workload_name(a), "frames_per_gpu": F, "H": H, "W": W, "channels": C,
+                   "in_dtype": a.dtype, "out_dtype": "i32", "l2": "inputs (7.46 GB at HD int32) larger than L2; no flush",
+                   "parallelism": f"frame-sharded x{world} (no data-path collective)",
+                   "kernel": {"1": "fused_tma_kernel", "2": "fused_generic_kernel"}[str(plan["kernel"])],
+                   "plan": plan},
+        "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s", "frac": achieved / peak,
+                     "traffic": traffic, "peak_source": peak_src,
+                     "algorithmic_bytes_per_launch": bpf * F,
+                     "avg_launch_ms": avg_launch_s * 1000.0, "min_launch_ms": min(launch_ms)},
+        "gpu_launches": a.steps,
+        "clocks": clk.summary(),
+    }
+    if e2e is not None:
+        line["e2e"] = e2e
+    if world > 1 and cs_all is not None:
+        line["gathered_checksums"] = int(cs_all.size)
+    if world == 1 and not a.no_cpu_baseline:
+        fps, info = cpu_baseline(a, gpu_cs=cs.cpu().view(torch.int64).numpy().view(np.uint64), frame0=frame0)
+        line["cpu_baseline"] = {"value": fps, "unit": "frames/s", "cores": info["cores"], "kind": "oracle",
+                                "sample": info["sample"], "parity_sample_ok": info.get("parity_sample_ok")}
+    print(json.dumps(line), flush=True)
+    if world > 1:
+        dist.destroy_process_group()
+
+
+if __name__ == "__main__":
+    main()

@@ -1,0 +1,240 @@
+/*
+ * aol.h -- C ABI of the B200 (sm_100a) ArrayOL downscaler library (libaol.so).
+ *
+ * What it computes: the data-parallel hot path of Guo et al., "Harnessing the
+ * Power of GPUs without Losing Abstractions in SaC and ArrayOL" (HIPS 2011),
+ * /root/reference/PAPER.md ("P:Lnnn" = line nnn).  The paper's running
+ * example is a two-stage HD->SD video downscaler (Fig. 2; task
+ * graph Fig. 3) whose stages are ArrayOL repetitions connected by
+ * tilers (Section IV):
+ *
+ *   pattern element  e(r, i) = (o + P.r + F.i) mod s_array
+ *   horizontal filter: pattern {11} every 8 columns -> 3 outputs   (Fig. 10)
+ *   vertical filter:   pattern {12} every 9 rows    -> 4 outputs   (reading Z1)
+ *   task: tile[k] = tmp/6 - tmp%6, tmp = 6-tap window sum          (Fig. 5)
+ *
+ * Conventions for every entry point:
+ *  - Device pointers ("d_") are owned by the caller (e.g. PyTorch); the library
+ *    allocates no device memory and holds no global state other than a
+ *    thread-local error string, so it is re-entrant.
+ *  - Device calls are stream-ordered on the given stream and return after
+ *    launch (asynchronous).  Kernel faults surface at the caller's next sync.
+ *  - Errors are returned synchronously as aol_status_t for invalid arguments,
+ *    shapes, dtypes, alignment, and launch failures; aol_last_error() then
+ *    holds a message.  On error nothing has been enqueued.
+ *  - Integer arithmetic is exact: results are bit-identical to the CPU oracle.
+ *  - Arrays are dense row-major; a batch of frames is planar
+ *    [frames][channels][H][W] (reading Z8: one plane per colour channel,
+ *    P:L671-675).
+ */
+#ifndef AOL_H
+#define AOL_H
+
+#include <stddef.h>
+#include <stdint.h>
+
+#include <cuda_runtime_api.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+#define AOL_VERSION 100 /* 1.0.0 */
+
+#if defined(__GNUC__)
+#define AOL_API __attribute__((visibility("default")))
+#else
+#define AOL_API
+#endif
+#define AOL_MAX_RANK 8
+
+typedef enum {
+    AOL_OK = 0,
+    AOL_E_INVALID = -1,   /* null pointer, rank or extent out of range, bad enum        */
+    AOL_E_SHAPE = -2,     /* W % 8 != 0, H % 9 != 0, or a shape the call cannot pave     */
+    AOL_E_DTYPE = -3,     /* element type not supported by this entry point              */
+    AOL_E_ALIGN = -4,     /* pointer not 16-byte aligned (TMA / vector access)          */
+    AOL_E_WORKSPACE = -5, /* workspace missing or too small                              */
+    AOL_E_RANGE = -6,     /* index arithmetic would overflow int64                       */
+    AOL_E_CUDA = -7       /* CUDA runtime / driver error (message in aol_last_error())   */
+} aol_status_t;
+
+typedef enum {
+    AOL_U8 = 1, AOL_I16 = 2, AOL_I32 = 3, AOL_I64 = 4, /* typed elements            */
+    AOL_RAW8 = 5, AOL_RAW16 = 6, AOL_RAW32 = 7, AOL_RAW64 = 8 /* raw bytes, same sizes */
+} aol_dtype_t;
+
+typedef enum {
+    AOL_SCATTER_FAST = 0,      /* caller asserts the output tiler is injective (ArrayOL single
+                                  assignment); one pass                             */
+    AOL_SCATTER_SEQUENTIAL = 1 /* Fig. 6 semantics: the LAST (r, i) in row-major
+                                  loop order wins on collisions; needs a workspace              */
+} aol_scatter_mode_t;
+
+/* ArrayOL tiler record (Fig. 10; Section IV).
+ * Shapes are extents > 0.  Matrices are row-major [array_dim][column]:
+ * paving[a][j] multiplies repetition index r_j, fitting[a][k] multiplies
+ * pattern index i_k (reading Z6: the paper prints matrices by columns; Fig. 11
+ * P:L720-725 pins the orientation).  origin and all matrix entries may be
+ * negative; the modulo is Euclidean, giving [0, s) (reading Z4).
+ * rep_rank / pattern_rank may be 0 (a single repetition / a scalar pattern). */
+typedef struct {
+    int32_t array_rank, rep_rank, pattern_rank; /* 1..8, 0..8, 0..8 */
+    int64_t array_shape[AOL_MAX_RANK];
+    int64_t rep_shape[AOL_MAX_RANK];
+    int64_t pattern_shape[AOL_MAX_RANK];
+    int64_t origin[AOL_MAX_RANK];
+    int64_t paving[AOL_MAX_RANK][AOL_MAX_RANK];
+    int64_t fitting[AOL_MAX_RANK][AOL_MAX_RANK];
+} aol_tiler_t;
+
+typedef enum {
+    AOL_PRESET_H_IN = 0,  /* Fig. 10 input tiler:  array {H,W}, pattern {11}, F=(0,1)^T, P=diag(1,8), rep {H,W/8} */
+    AOL_PRESET_H_OUT = 1, /* Fig. 10 output tiler: array {H,3W/8}, pattern {3}, F=(0,1)^T, P=diag(1,3), rep {H,W/8} */
+    AOL_PRESET_V_IN = 2,  /* reading Z1: array {H,W}, pattern {12}, F=(1,0)^T, P=diag(9,1), rep {H/9,W}            */
+    AOL_PRESET_V_OUT = 3  /* reading Z1: array {4H/9,W}, pattern {4}, F=(1,0)^T, P=diag(4,1), rep {H/9,W}           */
+} aol_preset_t;
+
+/* Optional launch tuning for aol_downscale_frame_ex (all zero = automatic). */
+typedef struct {
+    int32_t ctas_per_sm;    /* resident CTAs per SM for the fused kernel (1 or 2), 0 = auto     */
+    int32_t stages;         /* TMA ring depth in 3-row stages, 0 = as many as fit              */
+    int32_t bands_per_unit; /* 9-row bands per work unit, 0 = auto (balance waves vs halo)     */
+    int32_t kernel;         /* 0 = auto, 1 = TMA fused kernel (error if shape unsupported),
+                               2 = generic fused kernel (any W%8==0, H%9==0)                   */
+} aol_launch_opts_t;
+
+/* The launch configuration aol_downscale_frame_ex would use (for reports/tests). */
+typedef struct {
+    int32_t kernel;          /* 1 = TMA fused, 2 = generic fused                      */
+    int32_t grid, block;     /* CTAs, threads per CTA                                 */
+    int32_t smem_bytes;      /* dynamic shared memory per CTA                         */
+    int32_t stages;          /* TMA ring depth (kernel 1)                              */
+    int32_t bands_per_unit;  /* kernel 1                                               */
+    int64_t units;           /* work units (kernel 1)                                  */
+    int32_t ctas_per_sm;     /* kernel 1                                               */
+    int32_t num_sms;
+} aol_plan_t;
+
+/* ------------------------------------------------------------------ misc */
+
+/* Library version (AOL_VERSION). Never fails. */
+AOL_API int aol_version(void);
+
+/* Thread-local message describing the last error on this thread ("" if none).
+ * The pointer stays valid until the next aol_* call on the same thread. */
+AOL_API const char* aol_last_error(void);
+
+/* ------------------------------------------------------- tiler descriptors */
+
+/* Fill *out with the paper's tiler `which` for one plane.  H_IN/H_OUT take the
+ * input plane H x W (W % 8 == 0); V_IN/V_OUT take the intermediate plane
+ * H x W (H % 9 == 0).  Host only.  AOL_E_INVALID / AOL_E_SHAPE on bad input. */
+AOL_API aol_status_t aol_tiler_preset(aol_preset_t which, int64_t H, int64_t W, aol_tiler_t* out);
+
+/* Check ranks, extents, and that every index computation fits in int64.
+ * Host only.  Returns AOL_OK, AOL_E_INVALID or AOL_E_RANGE. */
+AOL_API aol_status_t aol_tiler_validate(const aol_tiler_t* t);
+
+/* *injective = 1 if no two (r, i) pairs address the same array element
+ * (brute force over the repetition x pattern space; a test helper meant for
+ * small descriptors).  Host only. */
+AOL_API aol_status_t aol_tiler_is_injective(const aol_tiler_t* t, int* injective);
+
+/* --------------------------------------------------- generic gather/scatter */
+
+/* Input tiler (Fig. 4; Section IV):
+ *   d_tiles[r][i] = d_array[(o + P.r + F.i) mod s]
+ * d_array: device, array_shape row-major, element type el (size 1/2/4/8 B).
+ * d_tiles: device, [rep_shape..., pattern_shape...] row-major, same element type.
+ * Both must be aligned to the element size.  Async on s. */
+AOL_API aol_status_t aol_tiler_gather(const aol_tiler_t* t, aol_dtype_t el, const void* d_array, void* d_tiles,
+                              cudaStream_t s);
+
+/* Bytes of device workspace aol_tiler_scatter needs in SEQUENTIAL mode
+ * (8 bytes per array element; 0 for a NULL/invalid tiler). */
+AOL_API size_t aol_tiler_scatter_workspace_bytes(const aol_tiler_t* t);
+
+/* Output tiler (Fig. 6; modarray): d_array[(o+P.r+F.i) mod s] = d_tiles[r][i],
+ * in place -- elements no (r, i) addresses keep their value.
+ * FAST: caller asserts injectivity (ArrayOL single assignment); collisions are
+ * then unspecified.  SEQUENTIAL: Fig. 6's loop order, the last writer wins;
+ * d_workspace must hold aol_tiler_scatter_workspace_bytes(t) bytes (it is
+ * overwritten).  Async on s. */
+AOL_API aol_status_t aol_tiler_scatter(const aol_tiler_t* t, aol_dtype_t el, const void* d_tiles, void* d_array,
+                               aol_scatter_mode_t mode, void* d_workspace, size_t ws_bytes, cudaStream_t s);
+
+/* ------------------------------------------------------------- the filters */
+
+/* Horizontal filter alone (the SaC/GASPARD2 "HorizontalFilter", Fig. 10 tilers
+ * + Fig. 5 task): d_in int32 [planes][H][W] -> d_out int32 [planes][H][3W/8].
+ * W % 8 == 0 else AOL_E_SHAPE.  Pointers 16-byte aligned.  Async on s. */
+AOL_API aol_status_t aol_downscale_h(const int32_t* d_in, int32_t* d_out, int64_t planes, int64_t H, int64_t W,
+                             cudaStream_t s);
+
+/* Vertical filter alone (reading Z1/Z2): d_in int32 [planes][H][W] ->
+ * d_out int32 [planes][4H/9][W].  H % 9 == 0 else AOL_E_SHAPE.  Async on s. */
+AOL_API aol_status_t aol_downscale_v(const int32_t* d_in, int32_t* d_out, int64_t planes, int64_t H, int64_t W,
+                             cudaStream_t s);
+
+/* The fused downscaler (hf -> vf of Fig. 3 in one kernel, the intermediate
+ * never touches HBM -- the hand-written analogue of SaC's WITH-loop folding,
+ * P:L528-546): d_in [frames][channels][H][W] -> d_out int32
+ * [frames][channels][4H/9][3W/8], H filter first (Fig. 2).
+ * in_dtype: AOL_I32 (values must lie in (-2^27, 2^27), reading Z12) or AOL_U8
+ * (8-bit samples).  d_frame_checksums: nullable device u64 [frames],
+ * overwritten with  sum (u64)(u32)Z[n][c][y][x] * (1 + (c*Ho + y)*Wo + x)  mod 2^64.
+ * frames == 0 is a no-op.  d_in/d_out 16-byte aligned.  Async on s. */
+AOL_API aol_status_t aol_downscale_frame(const void* d_in, aol_dtype_t in_dtype, int32_t* d_out, int64_t frames,
+                                 int64_t channels, int64_t H, int64_t W, uint64_t* d_frame_checksums,
+                                 cudaStream_t s);
+
+/* Same, with explicit launch options (NULL = automatic). */
+AOL_API aol_status_t aol_downscale_frame_ex(const void* d_in, aol_dtype_t in_dtype, int32_t* d_out, int64_t frames,
+                                    int64_t channels, int64_t H, int64_t W, uint64_t* d_frame_checksums,
+                                    const aol_launch_opts_t* opts, cudaStream_t s);
+
+/* Report the launch aol_downscale_frame_ex would make on the current device. */
+AOL_API aol_status_t aol_downscale_frame_plan(aol_dtype_t in_dtype, int64_t frames, int64_t channels, int64_t H,
+                                      int64_t W, const aol_launch_opts_t* opts, aol_plan_t* out);
+
+/* Per-frame checksum of an existing output batch (for the unfused paths):
+ * d_out int32 [frames][channels][Ho][Wo] -> d_checksums u64 [frames] (overwritten). */
+AOL_API aol_status_t aol_frame_checksum(const int32_t* d_out, int64_t frames, int64_t channels, int64_t Ho, int64_t Wo,
+                                uint64_t* d_checksums, cudaStream_t s);
+
+/* ------------------------------------------------- host-streamed end to end */
+
+/* Device workspace aol_downscale_frame_host needs for chunks of chunk_frames frames. */
+AOL_API size_t aol_downscale_frame_host_workspace_bytes(aol_dtype_t in_dtype, int64_t chunk_frames, int64_t channels,
+                                                int64_t H, int64_t W);
+
+/* The downscaler fed from and drained to HOST memory (the paper's runtime loop:
+ * H2D, filters, D2H per frame, Table I), pipelined in chunks of
+ * chunk_frames frames over three caller streams: s_h2d copies chunk k+1 in while
+ * s_compute downscales chunk k and s_d2h copies chunk k-1 out.
+ * h_in / h_out / h_frame_checksums: host buffers (pinned memory gives overlap;
+ * pageable memory works but serialises).  d_workspace: device, at least
+ * aol_downscale_frame_host_workspace_bytes(...) bytes.  BLOCKING: returns when
+ * h_out (and h_frame_checksums, nullable) are complete. */
+AOL_API aol_status_t aol_downscale_frame_host(const void* h_in, aol_dtype_t in_dtype, int32_t* h_out, int64_t frames,
+                                      int64_t channels, int64_t H, int64_t W, uint64_t* h_frame_checksums,
+                                      int64_t chunk_frames, void* d_workspace, size_t ws_bytes,
+                                      cudaStream_t s_h2d, cudaStream_t s_compute, cudaStream_t s_d2h);
+
+/* ------------------------------------------- synthetic input (test support) */
+
+/* Fill d_out [nframes][channels][H][W] with the counter-based synthetic frames
+ * of synth/ (the seeded generator shared with the oracle side; it stands in
+ * for the paper's OpenCV FrameGenerator):
+ *   u = splitmix64(seed*0x9E3779B97F4A7C15 + (((frame0+n)*channels + c)*H + y)*W + x)
+ *   kind 0 uniform u>>56 | 1 dark u>>61 | 2 signed (u>>37) - 2^26 | 3 ramp x | 4 constant value
+ * out_dtype AOL_I32 or AOL_U8 (kinds whose values fit).  Async on s. */
+AOL_API aol_status_t aol_synth_frames(uint64_t seed, int64_t frame0, int64_t nframes, int64_t channels, int64_t H,
+                              int64_t W, int32_t kind, int32_t value, aol_dtype_t out_dtype, void* d_out,
+                              cudaStream_t s);
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* AOL_H */

@@ -1,0 +1,268 @@
+"""B200-native ArrayOL downscaler (Guo et al., HIPS 2011) -- Python binding.
+
+Thin marshalling over the C ABI of ``include/aol.h`` (``libaol.so``): every
+step of the path runs in the library's sm_100a kernels; PyTorch only supplies
+device memory and the current CUDA stream.  There is no CPU fallback -- if the
+extension is missing, importing an entry point raises.
+
+Paper citations: tiler semantics Section IV
+(P:L292-319), SaC tiler functions Fig. 4-7, the downscaler
+tilers Fig. 10, the task Fig. 5.
+"""
+from __future__ import annotations
+
+import ctypes
+from typing import Optional, Sequence
+
+import torch
+
+from . import _lib
+from ._lib import (AolError, I16, I32, I64, PRESET_H_IN, PRESET_H_OUT, PRESET_V_IN, PRESET_V_OUT, RAW8, RAW16,
+                   RAW32, RAW64, SCATTER_FAST, SCATTER_SEQUENTIAL, U8, aol_launch_opts_t, aol_plan_t,
+                   aol_tiler_t, check, lib)
+
+__all__ = [
+    "AolError", "version", "make_tiler", "tiler_preset", "tiler_validate", "tiler_is_injective",
+    "tiler_gather", "tiler_scatter", "downscale_h", "downscale_v", "downscale_frame", "downscale_frame_plan",
+    "frame_checksum", "downscale_frame_host", "synth_frames", "library_path",
+    "PRESET_H_IN", "PRESET_H_OUT", "PRESET_V_IN", "PRESET_V_OUT", "SYNTH_KINDS",
+]
+
+SYNTH_KINDS = {"uniform": 0, "dark": 1, "signed": 2, "ramp": 3, "constant": 4}
+library_path = _lib.LIB_PATH
+
+_TYPED = {torch.uint8: U8, torch.int16: I16, torch.int32: I32, torch.int64: I64}
+_RAW = {1: RAW8, 2: RAW16, 4: RAW32, 8: RAW64}
+
+
+def _dtype_code(t: torch.Tensor) -> int:
+    if t.dtype in _TYPED:
+        return _TYPED[t.dtype]
+    es = t.element_size()
+    if es not in _RAW:
+        raise TypeError(f"unsupported element size {es}")
+    return _RAW[es]
+
+
+def _stream(stream: Optional[torch.cuda.Stream]) -> ctypes.c_void_p:
+    s = stream if stream is not None else torch.cuda.current_stream()
+    return ctypes.c_void_p(s.cuda_stream)
+
+
+def _dev(t: torch.Tensor, name: str) -> ctypes.c_void_p:
+    if not isinstance(t, torch.Tensor) or not t.is_cuda:
+        raise ValueError(f"{name} must be a CUDA tensor")
+    if not t.is_contiguous():
+        raise ValueError(f"{name} must be contiguous")
+    return ctypes.c_void_p(t.data_ptr())
+
+
+def version() -> int:
+    return int(lib().aol_version())
+
+
+# ------------------------------------------------------------------ tilers
+
+def make_tiler(array_shape: Sequence[int], rep_shape: Sequence[int], pattern_shape: Sequence[int],
+               origin: Optional[Sequence[int]] = None, paving=None, fitting=None) -> aol_tiler_t:
+    """ArrayOL tiler (Fig. 10 record): paving is [array_rank][rep_rank], fitting [array_rank][pattern_rank]."""
+    t = aol_tiler_t()
+    t.array_rank, t.rep_rank, t.pattern_rank = len(array_shape), len(rep_shape), len(pattern_shape)
+    for k, v in enumerate(array_shape):
+        t.array_shape[k] = int(v)
+    for k, v in enumerate(rep_shape):
+        t.rep_shape[k] = int(v)
+    for k, v in enumerate(pattern_shape):
+        t.pattern_shape[k] = int(v)
+    for a in range(len(array_shape)):
+        t.origin[a] = int(origin[a]) if origin is not None else 0
+        for j in range(len(rep_shape)):
+            t.paving[a][j] = int(paving[a][j]) if paving is not None else 0
+        for k in range(len(pattern_shape)):
+            t.fitting[a][k] = int(fitting[a][k]) if fitting is not None else 0
+    return t
+
+
+def _shapes(t: aol_tiler_t):
+    return (tuple(t.array_shape[k] for k in range(t.array_rank)),
+            tuple(t.rep_shape[k] for k in range(t.rep_rank)),
+            tuple(t.pattern_shape[k] for k in range(t.pattern_rank)))
+
+
+def tiler_preset(which: int, H: int, W: int) -> aol_tiler_t:
+    t = aol_tiler_t()
+    check(lib().aol_tiler_preset(which, H, W, ctypes.byref(t)))
+    return t
+
+
+def tiler_validate(t: aol_tiler_t) -> None:
+    check(lib().aol_tiler_validate(ctypes.byref(t)))
+
+
+def tiler_is_injective(t: aol_tiler_t) -> bool:
+    v = ctypes.c_int(0)
+    check(lib().aol_tiler_is_injective(ctypes.byref(t), ctypes.byref(v)))
+    return bool(v.value)
+
+
+def tiler_gather(t: aol_tiler_t, array: torch.Tensor, out: Optional[torch.Tensor] = None,
+                 stream: Optional[torch.cuda.Stream] = None) -> torch.Tensor:
+    """tiles[r][i] = array[(o + P.r + F.i) mod s]  (Fig. 4); returns [rep..., pattern...]."""
+    arr, rep, pat = _shapes(t)
+    if tuple(array.shape) != arr:
+        raise ValueError(f"array shape {tuple(array.shape)} != tiler array shape {arr}")
+    if out is None:
+        out = torch.empty(rep + pat, dtype=array.dtype, device=array.device)
+    elif tuple(out.shape) != rep + pat or out.dtype != array.dtype:
+        raise ValueError("out has the wrong shape or dtype")
+    check(lib().aol_tiler_gather(ctypes.byref(t), _dtype_code(array), _dev(array, "array"), _dev(out, "out"),
+                                 _stream(stream)))
+    return out
+
+
+def tiler_scatter(t: aol_tiler_t, tiles: torch.Tensor, array: torch.Tensor, mode: str = "fast",
+                  workspace: Optional[torch.Tensor] = None, stream: Optional[torch.cuda.Stream] = None) -> torch.Tensor:
+    """array[(o + P.r + F.i) mod s] = tiles[r][i] in place (Fig. 6).  mode: 'fast' | 'sequential'."""
+    arr, rep, pat = _shapes(t)
+    if tuple(array.shape) != arr or tuple(tiles.shape) != rep + pat or tiles.dtype != array.dtype:
+        raise ValueError("tiles/array shapes or dtypes do not match the tiler")
+    m = {"fast": SCATTER_FAST, "sequential": SCATTER_SEQUENTIAL}[mode]
+    ws_ptr, ws_bytes = ctypes.c_void_p(0), 0
+    if m == SCATTER_SEQUENTIAL:
+        need = int(lib().aol_tiler_scatter_workspace_bytes(ctypes.byref(t)))
+        if workspace is None:
+            workspace = torch.empty(need, dtype=torch.uint8, device=array.device)
+        ws_ptr, ws_bytes = _dev(workspace, "workspace"), workspace.numel() * workspace.element_size()
+    check(lib().aol_tiler_scatter(ctypes.byref(t), _dtype_code(array), _dev(tiles, "tiles"),
+                                  _dev(array, "array"), m, ws_ptr, ws_bytes, _stream(stream)))
+    return array
+
+
+# ------------------------------------------------------------------ filters
+
+def _planes(x: torch.Tensor):
+    if x.dim() < 2:
+        raise ValueError("expected [..., H, W]")
+    H, W = x.shape[-2:]
+    planes = 1
+    for d in x.shape[:-2]:
+        planes *= d
+    return planes, H, W
+
+
+def downscale_h(x: torch.Tensor, out: Optional[torch.Tensor] = None,
+                stream: Optional[torch.cuda.Stream] = None) -> torch.Tensor:
+    """Horizontal filter: int32 [..., H, W] -> [..., H, 3W/8]."""
+    if x.dtype != torch.int32:
+        raise TypeError("downscale_h takes int32")
+    planes, H, W = _planes(x)
+    if out is None:
+        out = torch.empty(x.shape[:-1] + (3 * (W // 8),), dtype=torch.int32, device=x.device)
+    check(lib().aol_downscale_h(_dev(x, "x"), _dev(out, "out"), planes, H, W, _stream(stream)))
+    return out
+
+
+def downscale_v(y: torch.Tensor, out: Optional[torch.Tensor] = None,
+                stream: Optional[torch.cuda.Stream] = None) -> torch.Tensor:
+    """Vertical filter: int32 [..., H, W] -> [..., 4H/9, W]."""
+    if y.dtype != torch.int32:
+        raise TypeError("downscale_v takes int32")
+    planes, H, W = _planes(y)
+    if out is None:
+        out = torch.empty(y.shape[:-2] + (4 * (H // 9), W), dtype=torch.int32, device=y.device)
+    check(lib().aol_downscale_v(_dev(y, "y"), _dev(out, "out"), planes, H, W, _stream(stream)))
+    return out
+
+
+def _opts(opts) -> Optional[aol_launch_opts_t]:
+    if opts is None:
+        return None
+    o = aol_launch_opts_t()
+    for k, v in dict(opts).items():
+        setattr(o, k, int(v))
+    return o
+
+
+def downscale_frame(x: torch.Tensor, out: Optional[torch.Tensor] = None, checksums=None, opts=None,
+                    stream: Optional[torch.cuda.Stream] = None):
+    """Fused downscaler: x [frames][channels][H][W] (int32 or uint8) -> int32 [frames][channels][4H/9][3W/8].
+
+    checksums: None (skip), True (allocate), or a uint64/int64 CUDA tensor [frames].
+    Returns (out, checksums_or_None)."""
+    if x.dim() != 4:
+        raise ValueError("x must be [frames][channels][H][W]")
+    if x.dtype not in (torch.int32, torch.uint8):
+        raise TypeError("x must be int32 or uint8")
+    N, C, H, W = x.shape
+    if out is None:
+        out = torch.empty((N, C, 4 * (H // 9), 3 * (W // 8)), dtype=torch.int32, device=x.device)
+    cs = checksums
+    if cs is True:
+        cs = torch.empty(N, dtype=torch.uint64, device=x.device)
+    cs_ptr = _dev(cs, "checksums") if cs is not None else ctypes.c_void_p(0)
+    o = _opts(opts)
+    check(lib().aol_downscale_frame_ex(_dev(x, "x"), _TYPED[x.dtype], _dev(out, "out"), N, C, H, W, cs_ptr,
+                                       ctypes.byref(o) if o is not None else None, _stream(stream)))
+    return out, cs
+
+
+def downscale_frame_plan(frames: int, channels: int, H: int, W: int, dtype=torch.int32, opts=None) -> dict:
+    p = aol_plan_t()
+    o = _opts(opts)
+    check(lib().aol_downscale_frame_plan(_TYPED[dtype], frames, channels, H, W,
+                                         ctypes.byref(o) if o is not None else None, ctypes.byref(p)))
+    return {f: getattr(p, f) for f, _ in aol_plan_t._fields_}
+
+
+def frame_checksum(z: torch.Tensor, out: Optional[torch.Tensor] = None,
+                   stream: Optional[torch.cuda.Stream] = None) -> torch.Tensor:
+    """Per-frame checksum of an int32 [frames][channels][Ho][Wo] batch."""
+    N, C, Ho, Wo = z.shape
+    if out is None:
+        out = torch.empty(N, dtype=torch.uint64, device=z.device)
+    check(lib().aol_frame_checksum(_dev(z, "z"), N, C, Ho, Wo, _dev(out, "out"), _stream(stream)))
+    return out
+
+
+def host_workspace_bytes(chunk_frames: int, channels: int, H: int, W: int, dtype=torch.int32) -> int:
+    return int(lib().aol_downscale_frame_host_workspace_bytes(_TYPED[dtype], chunk_frames, channels, H, W))
+
+
+def downscale_frame_host(x: torch.Tensor, out: Optional[torch.Tensor] = None, checksums: bool = True,
+                         chunk_frames: int = 16, workspace: Optional[torch.Tensor] = None, streams=None,
+                         device=None):
+    """End-to-end from HOST memory (pinned for overlap): H2D, fused kernel, D2H, pipelined.
+    Blocking.  Returns (out_host, checksums_host_or_None)."""
+    if x.is_cuda:
+        raise ValueError("x must be a host tensor")
+    if not x.is_contiguous():
+        raise ValueError("x must be contiguous")
+    N, C, H, W = x.shape
+    device = torch.device(device if device is not None else "cuda")
+    if out is None:
+        out = torch.empty((N, C, 4 * (H // 9), 3 * (W // 8)), dtype=torch.int32, pin_memory=x.is_pinned())
+    cs = torch.empty(N, dtype=torch.uint64, pin_memory=x.is_pinned()) if checksums else None
+    chunk = max(1, min(chunk_frames, N))
+    need = host_workspace_bytes(chunk, C, H, W, x.dtype)
+    if workspace is None:
+        workspace = torch.empty(need, dtype=torch.uint8, device=device)
+    if streams is None:
+        streams = [torch.cuda.Stream(device=device) for _ in range(3)]
+    sp = [ctypes.c_void_p(s.cuda_stream) for s in streams]
+    check(lib().aol_downscale_frame_host(
+        ctypes.c_void_p(x.data_ptr()), _TYPED[x.dtype], ctypes.c_void_p(out.data_ptr()), N, C, H, W,
+        ctypes.c_void_p(cs.data_ptr()) if cs is not None else ctypes.c_void_p(0), chunk,
+        _dev(workspace, "workspace"), workspace.numel(), sp[0], sp[1], sp[2]))
+    return out, cs
+
+
+def synth_frames(seed: int, frame0: int, nframes: int, channels: int, H: int, W: int, kind: str = "uniform",
+                 value: int = 0, dtype=torch.int32, device=None, out: Optional[torch.Tensor] = None,
+                 stream: Optional[torch.cuda.Stream] = None) -> torch.Tensor:
+    """Synthetic frames on the device (same counter-based generator as synth/)."""
+    if out is None:
+        out = torch.empty((nframes, channels, H, W), dtype=dtype,
+                          device=device if device is not None else "cuda")
+    check(lib().aol_synth_frames(seed & 0xFFFFFFFFFFFFFFFF, frame0, nframes, channels, H, W, SYNTH_KINDS[kind],
+                                 value, _TYPED[out.dtype], _dev(out, "out"), _stream(stream)))
+    return out

