@@ -227,15 +227,23 @@ def main():
     import torch.distributed as dist
 
     import paper_conf_ipps_guortgbs11_b200 as aol
+    from paper_conf_ipps_guortgbs11_b200 import shard
 
-    torch.cuda.set_device(local_rank)
-    dev = torch.device("cuda", local_rank)
+    # one process per GPU; AOL_DIST_BACKEND=gloo (and several ranks per GPU) only for testing the
+    # multi-rank flow on a 1-GPU box -- the driver's runs use NCCL with one GPU per rank
+    gpu = local_rank % max(1, torch.cuda.device_count())
+    torch.cuda.set_device(gpu)
+    dev = torch.device("cuda", gpu)
+    backend = os.environ.get("AOL_DIST_BACKEND", "nccl")
     if world > 1:
-        dist.init_process_group("nccl", device_id=dev)
+        if backend == "nccl":
+            dist.init_process_group("nccl", device_id=dev)
+        else:
+            dist.init_process_group(backend)
     opts = json.loads(a.opts) if a.opts else None
 
     F, C, H, W = a.frames, a.channels, a.H, a.W
-    frame0 = rank * F
+    frame0, F = shard.weak_range(rank, world, F)
     tdtype = torch.int32 if a.dtype == "i32" else torch.uint8
     x = aol.synth_frames(a.seed, frame0, F, C, H, W, "uniform", dtype=tdtype, device=dev)
     z = torch.empty((F, C, 4 * (H // 9), 3 * (W // 8)), dtype=torch.int32, device=dev)
@@ -254,7 +262,7 @@ def main():
     if world > 1:
         dist.barrier()
     torch.cuda.synchronize(dev)
-    with ClockSampler(local_rank) as clk:
+    with ClockSampler(gpu) as clk:
         t_begin.record(stream)
         for i in range(a.steps):
             starts[i].record(stream)
@@ -267,15 +275,9 @@ def main():
     elapsed_ms = t_begin.elapsed_time(t_end)
     launch_ms = [s.elapsed_time(e) for s, e in zip(starts, ends)]
 
-    # max over ranks (NCCL), and gather per-rank checksums + timings (the only cross-GPU traffic)
-    t = torch.tensor([elapsed_ms], dtype=torch.float64, device=dev)
-    cs_all = None
-    if world > 1:
-        dist.all_reduce(t, op=dist.ReduceOp.MAX)
-        gathered = torch.empty(world * F, dtype=torch.int64, device=dev)
-        dist.all_gather_into_tensor(gathered, cs.view(torch.int64))
-        cs_all = gathered.cpu().numpy().view(np.uint64)
-    max_ms = float(t.item())
+    # max over ranks (NCCL), and gather per-rank checksums: the only cross-GPU traffic
+    max_ms, cs_all_t = shard.gather_results(cs if backend == "nccl" else cs.cpu(), elapsed_ms)
+    cs_all = cs_all_t.cpu().numpy().view(np.uint64) if world > 1 else None
 
     # e2e through the host-buffer C-ABI call
     e2e = None
@@ -294,7 +296,7 @@ def main():
             _, cs_h = aol.downscale_frame_host(x_host, out=z_host, chunk_frames=chunk, workspace=ws,
                                                streams=streams, device=dev)
         e2e_s = time.perf_counter() - t0
-        te = torch.tensor([e2e_s], dtype=torch.float64, device=dev)
+        te = torch.tensor([e2e_s], dtype=torch.float64, device=dev if backend == "nccl" else "cpu")
         if world > 1:
             dist.all_reduce(te, op=dist.ReduceOp.MAX)
         e2e_s = float(te.item())

@@ -102,7 +102,11 @@ typedef struct {
     int32_t bands_per_unit; /* 9-row bands per work unit, 0 = auto (balance waves vs halo)     */
     int32_t kernel;         /* 0 = auto, 1 = TMA fused kernel (error if shape unsupported),
                                2 = generic fused kernel (any W%8==0, H%9==0)                   */
+    int32_t flags;          /* bit 0 (AOL_FLAG_HALO_LAST): stream a unit's 3 halo rows after its
+                               own rows instead of first (tuning experiment; same results)    */
 } aol_launch_opts_t;
+
+#define AOL_FLAG_HALO_LAST 1
 
 /* The launch configuration aol_downscale_frame_ex would use (for reports/tests). */
 typedef struct {

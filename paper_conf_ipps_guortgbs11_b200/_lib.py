@@ -47,7 +47,8 @@ class aol_tiler_t(ctypes.Structure):
 
 class aol_launch_opts_t(ctypes.Structure):
     _fields_ = [("ctas_per_sm", ctypes.c_int32), ("stages", ctypes.c_int32),
-                ("bands_per_unit", ctypes.c_int32), ("kernel", ctypes.c_int32)]
+                ("bands_per_unit", ctypes.c_int32), ("kernel", ctypes.c_int32),
+                ("flags", ctypes.c_int32)]
 
 
 class aol_plan_t(ctypes.Structure):

@@ -53,7 +53,7 @@ aol_status_t device_info(DeviceInfo* out);
 // ---- launchers implemented in the .cu files (all validate nothing; callers do)
 struct FusedPlan {
     int kernel;  // 1 = TMA fused, 2 = generic fused
-    int grid, block, smem, stages, bands_per_unit, ctas_per_sm, num_sms, units_per_plane;
+    int grid, block, smem, stages, bands_per_unit, ctas_per_sm, num_sms, units_per_plane, flags;
     int64_t units;
 };
 

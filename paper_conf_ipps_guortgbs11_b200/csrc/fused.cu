@@ -12,9 +12,12 @@
 //
 // Design (B200, sm_100a):
 //  * Work unit = (plane, run of `bands_per_unit` 9-row bands).  A unit streams
-//    3*nb + 1 "triples" of full-width rows: its own 9*nb rows plus the 3 halo
-//    rows (the next band's first rows, or rows 0..2 for the last band -- the
-//    toroidal wrap of the V tiler).  Persistent CTAs walk units round-robin.
+//    3*nb + 1 "triples" of full-width rows: first the 3 halo rows (the next
+//    unit's first rows, or rows 0..2 for the plane's last band -- the toroidal
+//    wrap of the V tiler), then its own 9*nb rows.  Loading the halo first
+//    makes it coincide with the neighbouring CTA's read of the same rows (an
+//    L2 hit instead of a second HBM read).  Persistent CTAs walk units
+//    round-robin.
 //  * One producer warp issues 3-D TMA tile loads (box = 3 rows x W int32,
 //    SWIZZLE_128B) into an S-stage smem ring guarded by full/empty mbarriers.
 //  * Consumer thread r owns repetition r (8 input columns -> 3 Y columns): two
@@ -42,6 +45,12 @@ namespace {
 
 constexpr int kMaxStages = 16;
 constexpr int kMaxConsumers = 992;  // + 1 producer warp = 1024 threads
+// Output staging buffers (4 output rows each).  One suffices: the bulk store of a
+// band has long finished reading smem by the time the next band (3 triples
+// later) is emitted, and the saved space buys one more ring stage.
+constexpr int kOutBufs = 1;
+// Bytes of TMA loads to keep in flight per SM (see plan_fused).
+constexpr int kInflightBytesPerSM = 6 * 23552;
 
 __device__ __forceinline__ int32_t task_T(int32_t S) {
     // Fig. 5: tmp/6 - tmp%6 == 7*(tmp/6) - tmp for C truncating division.
@@ -65,6 +74,7 @@ struct FusedArgs {
     uint32_t stage_stride;  // stage_bytes rounded up to 1024 (swizzle atom)
     uint32_t out_bytes;     // 16*Wo  (4 output rows)
     int32_t n_consumer;     // consumer threads, multiple of 32
+    int32_t halo_last;      // 1: stream the halo triple after the unit's own rows
 };
 
 // Byte offset of 16-byte chunk `chunk` (0..7) of 128-byte line `line` under SWIZZLE_128B
@@ -73,14 +83,14 @@ __device__ __forceinline__ uint32_t swz(uint32_t line, uint32_t chunk) {
     return (line << 7) | (((chunk ^ line) & 7u) << 4);
 }
 
-template <bool kChecksum, int kMaxThreads>
-__global__ void __launch_bounds__(kMaxThreads, 1)
+template <bool kChecksum, int kMaxThreads, int kMinBlocks>
+__global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
     fused_tma_kernel(const __grid_constant__ CUtensorMap tmap, const FusedArgs a) {
     extern __shared__ uint8_t smem_raw[];
     uint8_t* smem = reinterpret_cast<uint8_t*>((reinterpret_cast<uintptr_t>(smem_raw) + 1023) & ~uintptr_t(1023));
     uint8_t* stage_base = smem;
     int32_t* outbuf = reinterpret_cast<int32_t*>(smem + size_t(a.stages) * a.stage_stride);
-    uint64_t* full = reinterpret_cast<uint64_t*>(smem + size_t(a.stages) * a.stage_stride + 2 * a.out_bytes);
+    uint64_t* full = reinterpret_cast<uint64_t*>(smem + size_t(a.stages) * a.stage_stride + kOutBufs * a.out_bytes);
     uint64_t* empty = full + a.stages;
 
     const int tid = threadIdx.x;
@@ -106,13 +116,17 @@ __global__ void __launch_bounds__(kMaxThreads, 1)
                 const int32_t b1 = min(b0 + a.bands_per_unit, a.nbands);
                 const int32_t ntrip = 3 * (b1 - b0) + 1;
                 const int32_t row0 = int32_t(plane) * a.H;
-                int32_t trip = 3 * b0;
+                // halo triple first: rows 9*b1 .. 9*b1+2 (mod H -- the V tiler's toroidal wrap for the
+                // last band).  They are the first rows of the NEXT unit, which a neighbouring CTA
+                // streams at the same moment, so the second read hits L2 instead of HBM.
+                const int32_t halo = (3 * b1 == a.triples_per_plane) ? 0 : 3 * b1;
                 for (int32_t t = 0; t < ntrip; ++t) {
+                    const int32_t trip = a.halo_last ? (t == ntrip - 1 ? halo : 3 * b0 + t)
+                                                     : (t == 0 ? halo : 3 * b0 + t - 1);
                     ptx::mbar_wait(&empty[s], ph ^ 1u);
                     ptx::mbar_arrive_expect_tx(&full[s], a.stage_bytes);
                     ptx::tma_load_3d(stage_base + size_t(s) * a.stage_stride, &tmap, &full[s], 0, 0,
                                      row0 + 3 * trip);
-                    if (++trip == a.triples_per_plane) trip = 0;  // halo of the last band wraps (mod H)
                     if (++s == a.stages) {
                         s = 0;
                         ph ^= 1u;
@@ -133,6 +147,7 @@ __global__ void __launch_bounds__(kMaxThreads, 1)
     const uint32_t segn = uint32_t(rn) >> 2, chn = (uint32_t(rn) & 3u) << 1;
     const uint32_t segs = uint32_t(a.segs);
     const int Wo = a.Wo;
+    const uint32_t stage_s32 = ptx::smem_u32(stage_base);
 
     int s = 0;
     uint32_t ph = 0;
@@ -146,22 +161,63 @@ __global__ void __launch_bounds__(kMaxThreads, 1)
         const int32_t chan = int32_t(plane % a.channels);
         uint64_t csacc = 0;
 
-        int32_t A0[3], A1[3], A2[3], A3[3];
+        int32_t A0[3], A1[3], A2[3], A3[3];   // running V window sums of the current band
+        int32_t Hr9[3], Hr911[3];             // halo: Y row 9 and rows 9..11 of the unit's last band
 #pragma unroll
-        for (int m = 0; m < 3; ++m) A0[m] = A1[m] = A2[m] = A3[m] = 0;
+        for (int m = 0; m < 3; ++m) A0[m] = A1[m] = A2[m] = A3[m] = Hr9[m] = Hr911[m] = 0;
+
+        // Band `band` is complete once rows 9..11 of its pattern are known: z = T(window sums).
+        auto emit = [&](int32_t band, const int32_t* add9, const int32_t* add911) {
+            int32_t z[4][3];
+#pragma unroll
+            for (int m = 0; m < 3; ++m) {
+                z[0][m] = task_T(A0[m]);
+                z[1][m] = task_T(A1[m]);
+                z[2][m] = task_T(A2[m] + add9[m]);
+                z[3][m] = task_T(A3[m] + add911[m]);
+            }
+            if (tid == 0) ptx::bulk_wait_read<kOutBufs - 1>();   // the out buffer we reuse is free again
+            ptx::named_bar_sync(1, NC);
+            int32_t* ob = outbuf + (emit_idx % kOutBufs) * (a.out_bytes / 4);
+            if (active) {
+#pragma unroll
+                for (int k = 0; k < 4; ++k)
+#pragma unroll
+                    for (int m = 0; m < 3; ++m) ob[k * Wo + 3 * r + m] = z[k][m];
+            }
+            ptx::fence_proxy_async_smem();
+            ptx::named_bar_sync(1, NC);
+            if (tid == 0) {
+                int32_t* gz = a.Z + (size_t(plane) * a.Ho + size_t(4 * band)) * size_t(Wo);
+                ptx::bulk_store(gz, ob, a.out_bytes);   // 4 contiguous output rows
+                ptx::bulk_commit();
+            }
+            ++emit_idx;
+            if (kChecksum && active) {
+                const uint64_t w0 =
+                    1u + (uint64_t(chan) * a.Ho + uint64_t(4 * band)) * uint64_t(Wo) + uint64_t(3 * r);
+#pragma unroll
+                for (int k = 0; k < 4; ++k)
+#pragma unroll
+                    for (int m = 0; m < 3; ++m)
+                        csacc += uint64_t(uint32_t(z[k][m])) * (w0 + uint64_t(k) * Wo + uint64_t(m));
+            }
+        };
 
         int tau = 0;
-        for (int32_t t = 0; t < ntrip; ++t) {
+        for (int32_t ti = 0; ti < ntrip; ++ti) {
+            // logical triple index: 0 = halo, 1.. = the unit's own triples in order
+            const int32_t t = a.halo_last ? (ti == ntrip - 1 ? 0 : ti + 1) : ti;
             ptx::mbar_wait(&full[s], ph);
-            const uint8_t* sb = stage_base + size_t(s) * a.stage_stride;
+            const uint32_t sb = stage_s32 + uint32_t(s) * a.stage_stride;   // 32-bit shared address
 
             // ---- H stage on the 3 rows of this triple: y[row][col]
             int32_t y[3][3];
 #pragma unroll
             for (int rr = 0; rr < 3; ++rr) {
                 const uint32_t line = uint32_t(rr) * segs + seg;
-                const int4 q0 = *reinterpret_cast<const int4*>(sb + swz(line, ch0));
-                const int4 q1 = *reinterpret_cast<const int4*>(sb + swz(line, ch0 + 1));
+                const int4 q0 = ptx::lds128(sb + swz(line, ch0));
+                const int4 q1 = ptx::lds128(sb + swz(line, ch0 + 1));
                 const int32_t e = q0.x + q0.y;
                 const int32_t d = e + q0.z;                 // cols 8r..8r+2, the neighbour's halo
                 const int32_t q = q0.z + q0.w;
@@ -171,7 +227,7 @@ __global__ void __launch_bounds__(kMaxThreads, 1)
                 int32_t dn = __shfl_down_sync(0xffffffffu, d, 1);
                 if (fix) {
                     const uint32_t ln = uint32_t(rr) * segs + segn;
-                    const int4 qn = *reinterpret_cast<const int4*>(sb + swz(ln, chn));
+                    const int4 qn = ptx::lds128(sb + swz(ln, chn));
                     dn = qn.x + qn.y + qn.z;
                 }
                 y[rr][0] = task_T(e + qp);                  // window cols 0..5
@@ -185,45 +241,26 @@ __global__ void __launch_bounds__(kMaxThreads, 1)
                 ph ^= 1u;
             }
 
-            // ---- V stage: running sums of the 12-row pattern (starts 0,2,4,6)
+            if (t == 0) {   // the halo triple: keep what the last band needs from it
+#pragma unroll
+                for (int m = 0; m < 3; ++m) {
+                    Hr9[m] = y[0][m];
+                    Hr911[m] = y[0][m] + y[1][m] + y[2][m];
+                }
+                continue;
+            }
+
+            // ---- V stage: running sums of the 12-row pattern (windows start at rows 0,2,4,6)
             if (tau == 0) {
-                if (t > 0) {
-                    // rows 9,10,11 of the previous band complete it -> emit 4 output rows
-                    const int32_t band = b0 + t / 3 - 1;
-                    int32_t z[4][3];
+                if (t > 1) {
+                    // rows 0..2 of this band are rows 9..11 of the previous one: emit it
+                    int32_t r9[3], r911[3];
 #pragma unroll
                     for (int m = 0; m < 3; ++m) {
-                        z[0][m] = task_T(A0[m]);
-                        z[1][m] = task_T(A1[m]);
-                        z[2][m] = task_T(A2[m] + y[0][m]);
-                        z[3][m] = task_T(A3[m] + y[0][m] + y[1][m] + y[2][m]);
+                        r9[m] = y[0][m];
+                        r911[m] = y[0][m] + y[1][m] + y[2][m];
                     }
-                    if (tid == 0) ptx::bulk_wait_read<1>();     // out buffer (emit_idx & 1) is free
-                    ptx::named_bar_sync(1, NC);
-                    int32_t* ob = outbuf + (emit_idx & 1u) * (a.out_bytes / 4);
-                    if (active) {
-#pragma unroll
-                        for (int k = 0; k < 4; ++k)
-#pragma unroll
-                            for (int m = 0; m < 3; ++m) ob[k * Wo + 3 * r + m] = z[k][m];
-                    }
-                    ptx::fence_proxy_async_smem();
-                    ptx::named_bar_sync(1, NC);
-                    if (tid == 0) {
-                        int32_t* gz = a.Z + (size_t(plane) * a.Ho + size_t(4 * band)) * size_t(Wo);
-                        ptx::bulk_store(gz, ob, a.out_bytes);
-                        ptx::bulk_commit();
-                    }
-                    ++emit_idx;
-                    if (kChecksum && active) {
-                        const uint64_t w0 = 1u + (uint64_t(chan) * a.Ho + uint64_t(4 * band)) * uint64_t(Wo) +
-                                            uint64_t(3 * r);
-#pragma unroll
-                        for (int k = 0; k < 4; ++k)
-#pragma unroll
-                            for (int m = 0; m < 3; ++m)
-                                csacc += uint64_t(uint32_t(z[k][m])) * (w0 + uint64_t(k) * Wo + uint64_t(m));
-                    }
+                    emit(b0 + (t - 1) / 3 - 1, r9, r911);
                 }
 #pragma unroll
                 for (int m = 0; m < 3; ++m) {
@@ -249,6 +286,7 @@ __global__ void __launch_bounds__(kMaxThreads, 1)
             }
             if (++tau == 3) tau = 0;
         }
+        emit(b1 - 1, Hr9, Hr911);   // the unit's last band, completed by the halo rows
 
         if (kChecksum) {
 #pragma unroll
@@ -365,7 +403,7 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, const void* d_in, const int32_t* d
     DeviceInfo dev;
     aol_status_t st = device_info(&dev);
     if (st != AOL_OK) return st;
-    const aol_launch_opts_t o = opts ? *opts : aol_launch_opts_t{0, 0, 0, 0};
+    const aol_launch_opts_t o = opts ? *opts : aol_launch_opts_t{0, 0, 0, 0, 0};
     const int64_t planes = frames * channels;
     const int64_t Wo = 3 * (W / 8);
     *plan = FusedPlan{};
@@ -381,10 +419,17 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, const void* d_in, const int32_t* d
     if (tma_ok) {
         // per-CTA budget: share of the SM's smem, minus the 1 KB the runtime reserves per CTA
         int budget = std::min(dev.smem_optin, dev.smem_per_sm / ctas_per_sm - 1024);
-        int fixed = 2 * int(out_bytes) + 2 * kMaxStages * 8 + 1024;  // out buffers, barriers, align slack
+        int fixed = kOutBufs * int(out_bytes) + 2 * kMaxStages * 8 + 1024;  // out buffers, barriers, align slack
         stages = (budget - fixed) / int(stage_stride);
         stages = std::min(stages, kMaxStages);
-        if (o.stages > 0) stages = std::min(stages, o.stages);
+        if (o.stages > 0) {
+            stages = std::min(stages, o.stages);
+        } else {
+            // Measured on B200 (profiles/r01_*): throughput peaks at ~138 KB of TMA loads in flight per
+            // SM (6 HD row-triples); deeper rings are SLOWER (9 stages: -5%), shallower starve HBM.
+            const int target = (kInflightBytesPerSM / ctas_per_sm + int(stage_stride) / 2) / int(stage_stride);
+            stages = std::min(stages, std::max(2, target));
+        }
         if (stages < 2) tma_ok = false;
     }
     if (o.kernel == 1 && !tma_ok) {
@@ -421,8 +466,9 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, const void* d_in, const int32_t* d
         const int nc = int(((W / 8) + 31) / 32 * 32);
         plan->block = nc + 32;
         plan->stages = stages;
-        plan->smem = stages * int(stage_stride) + 2 * int(out_bytes) + 2 * stages * 8 + 1024;
+        plan->smem = stages * int(stage_stride) + kOutBufs * int(out_bytes) + 2 * stages * 8 + 1024;
         plan->ctas_per_sm = ctas_per_sm;
+        plan->flags = o.flags;
     } else {
         plan->kernel = 2;
         plan->block = 256;
@@ -489,10 +535,14 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
     a.stage_stride = (a.stage_bytes + 1023u) & ~1023u;
     a.out_bytes = uint32_t(16 * Wo);
     a.n_consumer = plan.block - 32;
+    a.halo_last = (plan.flags & AOL_FLAG_HALO_LAST) ? 1 : 0;
 
     // <=512 threads (W <= 3840): register budget for 1-2 CTAs/SM; wider rows need the 1024-thread build
-    auto k = plan.block <= 512 ? (d_cs ? fused_tma_kernel<true, 512> : fused_tma_kernel<false, 512>)
-                               : (d_cs ? fused_tma_kernel<true, 1024> : fused_tma_kernel<false, 1024>);
+    // register budget per residency: <=320 threads x 2 CTAs/SM, <=512 x 1, <=1024 x 1
+    auto k = (plan.block <= 320 && plan.ctas_per_sm >= 2)
+                 ? (d_cs ? fused_tma_kernel<true, 320, 2> : fused_tma_kernel<false, 320, 2>)
+             : plan.block <= 512 ? (d_cs ? fused_tma_kernel<true, 512, 1> : fused_tma_kernel<false, 512, 1>)
+                                 : (d_cs ? fused_tma_kernel<true, 1024, 1> : fused_tma_kernel<false, 1024, 1>);
     AOL_CUDA_TRY(cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, plan.smem));
     k<<<plan.grid, plan.block, plan.smem, s>>>(map, a);
     AOL_LAUNCH_CHECK("fused_tma_kernel");

@@ -79,6 +79,7 @@ def test_fused_vs_oracle(orc, shape, kernel):
 @pytest.mark.parametrize("opts", [
     {"bands_per_unit": 1}, {"bands_per_unit": 2}, {"bands_per_unit": 7}, {"bands_per_unit": 40},
     {"stages": 2}, {"stages": 3, "bands_per_unit": 5}, {"ctas_per_sm": 2}, {"ctas_per_sm": 2, "stages": 2},
+    {"flags": 1}, {"flags": 1, "bands_per_unit": 1, "stages": 2},
 ])
 def test_fused_launch_options(orc, opts):
     """Unit boundaries, ring wrap-around and CTA residency do not change results."""
