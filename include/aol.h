@@ -97,7 +97,7 @@ typedef enum {
 
 /* Optional launch tuning for aol_downscale_frame_ex (all zero = automatic). */
 typedef struct {
-    int32_t ctas_per_sm;    /* resident CTAs per SM for the fused kernel (1 or 2), 0 = auto     */
+    int32_t ctas_per_sm;    /* resident CTAs per SM for the fused kernel (1..8), 0 = auto       */
     int32_t stages;         /* TMA ring depth in 3-row stages, 0 = as many as fit              */
     int32_t bands_per_unit; /* 9-row bands per work unit, 0 = auto (balance waves vs halo)     */
     int32_t kernel;         /* 0 = auto, 1 = TMA fused kernel (error if shape unsupported),

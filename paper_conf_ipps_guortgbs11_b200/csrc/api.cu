@@ -121,6 +121,32 @@ aol_status_t make_tiler_dev(const aol_tiler_t* t, TilerDev* td) {
         for (int k = 0; k < t->pattern_rank; ++k) td->coef[a][t->rep_rank + k] = emod(t->fitting[a][k], s);
     }
     td->array_elems = stride;
+    // classify: which array dims can wrap, affine offsets, fast 32-bit division
+    td->linear = 1;
+    td->nowrap_mask = 0;
+    td->base = 0;
+    for (int a = 0; a < td->ra; ++a) {
+        __int128 mx = td->org[a];
+        for (int d = 0; d < td->nd; ++d) mx += __int128(td->coef[a][d]) * (td->ext[d] - 1);
+        if (mx < td->ashape[a]) td->nowrap_mask |= 1u << a;
+        else td->linear = 0;
+        td->base += td->org[a] * td->astride[a];
+    }
+    for (int d = 0; d < td->nd; ++d) {
+        int64_t l = 0;
+        for (int a = 0; a < td->ra; ++a) l += td->coef[a][d] * td->astride[a];
+        td->lin[d] = td->linear ? l : 0;
+    }
+    td->fast32 = total < (int64_t(1) << 31) ? 1 : 0;
+    for (int d = 0; d < td->nd; ++d) {
+        // n / ext == (umulhi(n, mul) + n) >> shift for n, ext < 2^31
+        uint32_t shift = 0;
+        while (shift < 32 && (uint64_t(1) << shift) < uint64_t(td->ext[d])) ++shift;
+        const uint64_t magic = ((uint64_t(1) << 32) * ((uint64_t(1) << shift) - uint64_t(td->ext[d]))) /
+                                   uint64_t(td->ext[d]) + 1;
+        td->fd_mul[d] = td->fast32 ? uint32_t(magic) : 0u;
+        td->fd_shift[d] = shift;
+    }
     return AOL_OK;
 }
 
@@ -154,7 +180,7 @@ aol_status_t frame_ex(const void* d_in, aol_dtype_t in_dtype, int32_t* d_out, in
     aol_status_t st = check_frame_args(d_in, in_dtype, d_out, frames, channels, H, W);
     if (st != AOL_OK) return st;
     if (frames == 0) return AOL_OK;
-    if (opts && (opts->ctas_per_sm < 0 || opts->ctas_per_sm > 2 || opts->stages < 0 || opts->bands_per_unit < 0 ||
+    if (opts && (opts->ctas_per_sm < 0 || opts->ctas_per_sm > 8 || opts->stages < 0 || opts->bands_per_unit < 0 ||
                  opts->kernel < 0 || opts->kernel > 2))
         return fail(AOL_E_INVALID, "launch options out of range");
     FusedPlan plan;

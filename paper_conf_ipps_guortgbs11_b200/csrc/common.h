@@ -72,11 +72,17 @@ aol_status_t launch_checksum(const int32_t* d_out, int64_t frames, int64_t per_f
 // Generic tiler: device-ready descriptor (coefficients reduced mod the array extents).
 struct TilerDev {
     int32_t ra, nd;             // array rank, combined (rep ++ pattern) rank
+    int32_t linear;             // 1: no coordinate can wrap -> offset is affine in the tile index
+    int32_t fast32;             // 1: total < 2^31 -> 32-bit magic-number division
+    uint32_t nowrap_mask;       // bit a: array dim a never wraps
     int64_t ext[2 * AOL_MAX_RANK];
     int64_t coef[AOL_MAX_RANK][2 * AOL_MAX_RANK];
     int64_t org[AOL_MAX_RANK];
     int64_t ashape[AOL_MAX_RANK];
     int64_t astride[AOL_MAX_RANK];
+    int64_t lin[2 * AOL_MAX_RANK];  // element offset per unit of combined index d (linear tilers)
+    int64_t base;                   // element offset of the origin
+    uint32_t fd_mul[2 * AOL_MAX_RANK], fd_shift[2 * AOL_MAX_RANK];
     int64_t total;              // rep elements * pattern elements
     int64_t array_elems;
 };

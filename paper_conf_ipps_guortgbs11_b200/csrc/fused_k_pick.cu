@@ -1,0 +1,18 @@
+// Dispatch between the separately compiled fused_tma_kernel instantiations.
+#include "fused_kernel.cuh"
+
+namespace aol {
+namespace fused {
+KernelFn tma_kernel_i32_cs(int block, int cps);
+KernelFn tma_kernel_i32_nocs(int block, int cps);
+KernelFn tma_kernel_u8_cs(int block, int cps);
+KernelFn tma_kernel_u8_nocs(int block, int cps);
+
+KernelFn tma_kernel_i32(bool checksum, int block, int cps) {
+    return checksum ? tma_kernel_i32_cs(block, cps) : tma_kernel_i32_nocs(block, cps);
+}
+KernelFn tma_kernel_u8(bool checksum, int block, int cps) {
+    return checksum ? tma_kernel_u8_cs(block, cps) : tma_kernel_u8_nocs(block, cps);
+}
+}  // namespace fused
+}  // namespace aol

@@ -1,0 +1,447 @@
+// fused.cu -- K-5: the fused HD->SD downscaler (hf -> vf of Fig. 3 in one kernel).
+//
+// What it computes: per plane X[H][W] (one colour channel)
+//   H stage  (Fig. 10 tilers P:L681-694, Fig. 5 task P:L435-446):
+//     Y[y][3r+k] = T( sum_{t<6} X[y][(8r + s_k + t) mod W] ),  s = (0,2,5)
+//   V stage  (reading Z1/Z2):
+//     Z[4b+k][x] = T( sum_{t<6} Y[(9b + 2k + t) mod H][x] )
+//   T(S) = S/6 - S%6 (C int semantics)  ==  7*(S/6) - S.
+// Y never touches HBM: the hand-written analogue of SaC's WITH-loop folding
+// (P:L528-546), in one launch instead of the 5 + 7 generator kernels
+// SaC-CUDA produced.
+//
+// Design (B200, sm_100a):
+//  * Work unit = (plane, run of `bands_per_unit` 9-row bands).  A unit streams
+//    3*nb + 1 "triples" of full-width rows: first the 3 halo rows (the next
+//    unit's first rows, or rows 0..2 for the plane's last band -- the toroidal
+//    wrap of the V tiler), then its own 9*nb rows.  Loading the halo first
+//    makes it coincide with the neighbouring CTA's read of the same rows (an
+//    L2 hit instead of a second HBM read).  Persistent CTAs walk units
+//    round-robin.
+//  * One producer warp fills an S-stage smem ring guarded by full/empty
+//    mbarriers.  int32 input: 3-D TMA tensor loads (box = 3 rows x W,
+//    SWIZZLE_128B).  uint8 input ("24-bit RGB"): 1-D TMA bulk copies of
+//    the contiguous 3-row triple.
+//  * Consumer thread r owns repetition r (8 input columns -> 3 Y columns).
+//    int32: two conflict-free LDS.128 per row (the 128B swizzle spreads the
+//    32-byte per-thread stride over all banks).  uint8: one LDS.64 per row and
+//    six DP4A byte-dot-products form the three 6-tap sums.  Either way ONE
+//    warp shuffle supplies the 3-column pattern overlap (pattern {11} vs paving
+//    step 8); lane 31 and the row-wrapping repetition read it from smem.
+//  * The V stage is a running register accumulation over the band's rows
+//    (4 outputs x 3 columns per thread), so every input row is read once.
+//  * Each finished band (4 output rows, contiguous in Z) is staged in smem and
+//    written by one 1-D TMA bulk store; the per-frame checksum is folded in
+//    registers and added with one atomic per warp per unit.
+#pragma once
+#include <cuda.h>
+#include <cuda_runtime.h>
+
+#include <cstdint>
+#include <type_traits>
+
+#include "ptx.cuh"
+
+namespace aol {
+namespace fused {
+
+
+constexpr int kMaxStages = 32;
+constexpr int kMaxConsumers = 992;  // + 1 producer warp = 1024 threads
+// Output staging buffers (4 output rows each).  One suffices: the bulk store of a
+// band has long finished reading smem by the time the next band (3 triples
+// later) is emitted, and the saved space buys one more ring stage.
+constexpr int kOutBufs = 1;
+// Bytes of TMA loads to keep in flight per SM.  Measured on B200
+// (profiles/r01_stage_sweep.jsonl): HD int32 throughput peaks at 6 row-triples
+// (138 KB) per SM; deeper rings are SLOWER (9 stages: -5%), shallower starve HBM.
+constexpr int kInflightBytesPerSM = 6 * 23552;
+
+__device__ __forceinline__ int32_t task_T(int32_t S) {
+    // Fig. 5: tmp/6 - tmp%6 == 7*(tmp/6) - tmp for C truncating division.
+    return 7 * (S / 6) - S;
+}
+
+// Same for 0 <= S < 98304 (sums of six 8-bit samples are <= 1530): S/6 == (S * 43691) >> 18 exactly
+// there without 32-bit overflow (43691 = (2^18 + 2) / 6; checked exhaustively in tests/test_abi.py).
+__device__ __forceinline__ int32_t task_T_nonneg(int32_t S) {
+    const int32_t q = int32_t((uint32_t(S) * 43691u) >> 18);
+    return 7 * q - S;
+}
+
+struct FusedArgs {
+    int32_t* Z;
+    uint64_t* cs;
+    const void* X;              // uint8 path: source of the 1-D bulk copies
+    int64_t nunits;
+    int32_t H, W, Ho, Wo;
+    int32_t channels;
+    int32_t reps;               // W/8  repetitions of the H tiler per row
+    int32_t segs;               // int32 path: W/32 128-byte segments per row
+    int32_t triples_per_plane;  // H/3
+    int32_t nbands;             // H/9
+    int32_t bands_per_unit;
+    int32_t units_per_plane;
+    int32_t stages;
+    uint32_t stage_bytes;   // bytes of one row triple (12W int32, 3W uint8)
+    uint32_t stage_stride;  // stage_bytes rounded up (1024 for the swizzle atom, 128 for uint8)
+    uint32_t out_bytes;     // 16*Wo  (4 output rows)
+    int32_t n_consumer;     // consumer threads, multiple of 32
+    int32_t halo_last;      // 1: stream the halo triple after the unit's own rows
+};
+
+// Byte offset of 16-byte chunk `chunk` (0..7) of 128-byte line `line` under SWIZZLE_128B
+// (chunk index XOR line index mod 8; stage buffers are 1024-byte aligned).
+__device__ __forceinline__ uint32_t swz(uint32_t line, uint32_t chunk) {
+    return (line << 7) | (((chunk ^ line) & 7u) << 4);
+}
+
+// Per-thread constants of the H stage (which repetition, where its bytes live).
+struct RepGeom {
+    uint32_t off0, off1;  // int32: swizzled offsets of the two chunks within a row's lines; uint8: 8r
+    uint32_t offn;        // neighbour repetition's first chunk / word
+    uint32_t seg, segn;   // int32: 128-byte segment of the repetition and of its neighbour
+    bool fix;             // read the neighbour from smem instead of the shuffle
+};
+
+// H stage of one input row: the three 6-tap window sums of repetition r, T() applied.
+template <typename Tin>
+__device__ __forceinline__ void h_row(uint32_t row_base, uint32_t rr, const RepGeom& g, uint32_t segs, uint32_t W,
+                                      int32_t& y0, int32_t& y1, int32_t& y2) {
+    if constexpr (std::is_same<Tin, int32_t>::value) {
+        const uint32_t line = rr * segs + g.seg;
+        const int4 q0 = ptx::lds128(row_base + swz(line, g.off0));
+        const int4 q1 = ptx::lds128(row_base + swz(line, g.off1));
+        const int32_t e = q0.x + q0.y;
+        const int32_t d = e + q0.z;                 // cols 8r..8r+2: the left neighbour's overlap
+        const int32_t q = q0.z + q0.w;
+        const int32_t p = q1.x + q1.y;
+        const int32_t f = q1.z + q1.w;
+        const int32_t qp = q + p;
+        int32_t dn = __shfl_down_sync(0xffffffffu, d, 1);
+        int4 qn = q0;   // lane 31 / wrapping repetition: neighbour chunk from smem (predicated, no branch)
+        ptx::lds128_if(qn, row_base + swz(rr * segs + g.segn, g.offn), g.fix);
+        dn = g.fix ? qn.x + qn.y + qn.z : dn;
+        y0 = task_T(e + qp);            // window cols 0..5
+        y1 = task_T(qp + f);            // window cols 2..7
+        y2 = task_T(q1.y + f + dn);     // window cols 5..10
+    } else {
+        // uint8 samples: bytes 0..7 of the repetition in two words; dp4a(x, m, c) = c + sum of the
+        // bytes of x selected by the 0/1 bytes of m (byte k = bits 8k..8k+7 = column 8r+k).
+        const uint32_t rowa = row_base + rr * W;
+        const uint2 v = ptx::lds64(rowa + g.off0);
+        uint32_t nw = __shfl_down_sync(0xffffffffu, v.x, 1);
+        ptx::lds32_if(nw, rowa + g.offn, g.fix);   // lane 31 / wrapping repetition (predicated)
+        const int32_t S0 = int32_t(__dp4a(v.x, 0x01010101u, __dp4a(v.y, 0x00000101u, 0u)));  // cols 0..5
+        const int32_t S1 = int32_t(__dp4a(v.x, 0x01010000u, __dp4a(v.y, 0x01010101u, 0u)));  // cols 2..7
+        const int32_t S2 = int32_t(__dp4a(v.y, 0x01010100u, __dp4a(nw, 0x00010101u, 0u)));   // cols 5..10
+        y0 = task_T_nonneg(S0);   // 8-bit samples: 0 <= S <= 1530
+        y1 = task_T_nonneg(S1);
+        y2 = task_T_nonneg(S2);
+    }
+}
+
+template <typename Tin, bool kChecksum, int kMaxThreads, int kMinBlocks>
+__global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
+    fused_tma_kernel(const __grid_constant__ CUtensorMap tmap, const FusedArgs a) {
+    constexpr bool kI32 = std::is_same<Tin, int32_t>::value;
+    extern __shared__ uint8_t smem_raw[];
+    uint8_t* smem = reinterpret_cast<uint8_t*>((reinterpret_cast<uintptr_t>(smem_raw) + 1023) & ~uintptr_t(1023));
+    uint8_t* stage_base = smem;
+    int32_t* outbuf = reinterpret_cast<int32_t*>(smem + size_t(a.stages) * a.stage_stride);
+    uint64_t* full = reinterpret_cast<uint64_t*>(smem + size_t(a.stages) * a.stage_stride + kOutBufs * a.out_bytes);
+    uint64_t* empty = full + a.stages;
+
+    const int tid = threadIdx.x;
+    const int NC = a.n_consumer;
+    if (tid == 0) {
+        for (int s = 0; s < a.stages; ++s) {
+            ptx::mbar_init(&full[s], 1);
+            ptx::mbar_init(&empty[s], NC / 32);
+        }
+        ptx::fence_mbar_init();
+    }
+    __syncthreads();
+
+    if (tid >= NC) {
+        // ------------------------------------------------ producer warp (TMA)
+        if (tid == NC) {
+            if (kI32) ptx::prefetch_tensormap(&tmap);
+            int s = 0;
+            uint32_t ph = 0;
+            for (int64_t u = blockIdx.x; u < a.nunits; u += gridDim.x) {
+                const int64_t plane = u / a.units_per_plane;
+                const int32_t b0 = int32_t(u - plane * a.units_per_plane) * a.bands_per_unit;
+                const int32_t b1 = min(b0 + a.bands_per_unit, a.nbands);
+                const int32_t ntrip = 3 * (b1 - b0) + 1;
+                const int64_t row0 = plane * a.H;
+                // halo triple: rows 9*b1 .. 9*b1+2 (mod H -- the V tiler's toroidal wrap for the last band)
+                const int32_t halo = (3 * b1 == a.triples_per_plane) ? 0 : 3 * b1;
+                for (int32_t t = 0; t < ntrip; ++t) {
+                    const int32_t trip = a.halo_last ? (t == ntrip - 1 ? halo : 3 * b0 + t)
+                                                     : (t == 0 ? halo : 3 * b0 + t - 1);
+                    ptx::mbar_wait_sleep(&empty[s], ph ^ 1u);   // suspended, not spinning, while the ring is full
+                    ptx::mbar_arrive_expect_tx(&full[s], a.stage_bytes);
+                    uint8_t* dst = stage_base + size_t(s) * a.stage_stride;
+                    if constexpr (kI32) {
+                        ptx::tma_load_3d(dst, &tmap, &full[s], 0, 0, int32_t(row0 + 3 * trip));
+                    } else {
+                        const uint8_t* src = static_cast<const uint8_t*>(a.X) + size_t(row0 + 3 * trip) * a.W;
+                        ptx::bulk_load(dst, src, a.stage_bytes, &full[s]);
+                    }
+                    if (++s == a.stages) {
+                        s = 0;
+                        ph ^= 1u;
+                    }
+                }
+            }
+        }
+        return;
+    }
+
+    // ---------------------------------------------------- consumer threads
+    const int lane = tid & 31;
+    const bool active = tid < a.reps;
+    const int r = active ? tid : a.reps - 1;        // repetition owned (clamped for idle lanes)
+    const int rn = (r + 1 == a.reps) ? 0 : r + 1;  // neighbour repetition (toroidal, Fig. 11 '% 1920')
+    RepGeom g;
+    g.fix = (lane == 31) || (r + 1 == a.reps);
+    if constexpr (kI32) {
+        g.seg = uint32_t(r) >> 2;
+        g.segn = uint32_t(rn) >> 2;
+        g.off0 = (uint32_t(r) & 3u) << 1;   // chunk indices within the 128-byte line
+        g.off1 = g.off0 + 1;
+        g.offn = (uint32_t(rn) & 3u) << 1;
+    } else {
+        g.seg = g.segn = 0;
+        g.off0 = 8u * uint32_t(r);
+        g.off1 = g.off0 + 4;
+        g.offn = 8u * uint32_t(rn);
+    }
+    const uint32_t segs = uint32_t(a.segs);
+    const uint32_t Wu = uint32_t(a.W);
+    const int Wo = a.Wo;
+    const uint32_t stage_s32 = ptx::smem_u32(stage_base);
+
+    int s = 0;
+    uint32_t ph = 0;
+    uint32_t emit_idx = 0;
+
+    for (int64_t u = blockIdx.x; u < a.nunits; u += gridDim.x) {
+        const int64_t plane = u / a.units_per_plane;
+        const int32_t b0 = int32_t(u - plane * a.units_per_plane) * a.bands_per_unit;
+        const int32_t b1 = min(b0 + a.bands_per_unit, a.nbands);
+        const int32_t ntrip = 3 * (b1 - b0) + 1;
+        const int32_t chan = int32_t(plane % a.channels);
+        uint64_t csacc = 0;
+
+        int32_t A0[3], A1[3], A2[3], A3[3];   // running V window sums of the current band
+        int32_t Hr9[3], Hr911[3];             // halo: Y row 9 and rows 9..11 of the unit's last band
+#pragma unroll
+        for (int m = 0; m < 3; ++m) A0[m] = A1[m] = A2[m] = A3[m] = Hr9[m] = Hr911[m] = 0;
+
+        // Band `band` is complete once rows 9..11 of its pattern are known: z = T(window sums).
+        auto emit = [&](int32_t band, const int32_t* add9, const int32_t* add911) {
+            int32_t z[4][3];
+#pragma unroll
+            for (int m = 0; m < 3; ++m) {
+                z[0][m] = task_T(A0[m]);
+                z[1][m] = task_T(A1[m]);
+                z[2][m] = task_T(A2[m] + add9[m]);
+                z[3][m] = task_T(A3[m] + add911[m]);
+            }
+            if (tid == 0) ptx::bulk_wait_read<kOutBufs - 1>();   // the out buffer we reuse is free again
+            ptx::named_bar_sync(1, NC);
+            const uint32_t ob = ptx::smem_u32(outbuf) + (emit_idx % kOutBufs) * a.out_bytes;
+            if (active) {
+#pragma unroll
+                for (int k = 0; k < 4; ++k)
+#pragma unroll
+                    for (int m = 0; m < 3; ++m) ptx::sts32(ob + 4u * uint32_t(k * Wo + 3 * r + m), z[k][m]);
+            }
+            ptx::fence_proxy_async_smem();
+            ptx::named_bar_sync(1, NC);
+            if (tid == 0) {
+                int32_t* gz = a.Z + (size_t(plane) * a.Ho + size_t(4 * band)) * size_t(Wo);
+                ptx::bulk_store(gz, outbuf + (emit_idx % kOutBufs) * (a.out_bytes / 4), a.out_bytes);   // 4 rows
+                ptx::bulk_commit();
+            }
+            ++emit_idx;
+            if (kChecksum && active) {
+                const uint64_t w0 =
+                    1u + (uint64_t(chan) * a.Ho + uint64_t(4 * band)) * uint64_t(Wo) + uint64_t(3 * r);
+#pragma unroll
+                for (int k = 0; k < 4; ++k)
+#pragma unroll
+                    for (int m = 0; m < 3; ++m)
+                        csacc += uint64_t(uint32_t(z[k][m])) * (w0 + uint64_t(k) * Wo + uint64_t(m));
+            }
+        };
+
+        int tau = 0;
+        for (int32_t ti = 0; ti < ntrip; ++ti) {
+            // logical triple index: 0 = halo, 1.. = the unit's own triples in order
+            const int32_t t = a.halo_last ? (ti == ntrip - 1 ? 0 : ti + 1) : ti;
+            ptx::mbar_wait_sleep(&full[s], ph);
+            const uint32_t sb = stage_s32 + uint32_t(s) * a.stage_stride;   // 32-bit shared address
+
+            // ---- H stage on the 3 rows of this triple: y[row][col]
+            int32_t y[3][3];
+#pragma unroll
+            for (int rr = 0; rr < 3; ++rr) h_row<Tin>(sb, uint32_t(rr), g, segs, Wu, y[rr][0], y[rr][1], y[rr][2]);
+            __syncwarp();
+            if (lane == 0) ptx::mbar_arrive(&empty[s]);
+            if (++s == a.stages) {
+                s = 0;
+                ph ^= 1u;
+            }
+
+            if (t == 0) {   // the halo triple: keep what the last band needs from it
+#pragma unroll
+                for (int m = 0; m < 3; ++m) {
+                    Hr9[m] = y[0][m];
+                    Hr911[m] = y[0][m] + y[1][m] + y[2][m];
+                }
+                continue;
+            }
+
+            // ---- V stage: running sums of the 12-row pattern (windows start at rows 0,2,4,6)
+            if (tau == 0) {
+                if (t > 1) {
+                    // rows 0..2 of this band are rows 9..11 of the previous one: emit it
+                    int32_t r9[3], r911[3];
+#pragma unroll
+                    for (int m = 0; m < 3; ++m) {
+                        r9[m] = y[0][m];
+                        r911[m] = y[0][m] + y[1][m] + y[2][m];
+                    }
+                    emit(b0 + (t - 1) / 3 - 1, r9, r911);
+                }
+#pragma unroll
+                for (int m = 0; m < 3; ++m) {
+                    A0[m] = y[0][m] + y[1][m] + y[2][m];   // rows 0..2 of window 0..5
+                    A1[m] = y[2][m];                        // row 2 of window 2..7
+                }
+            } else if (tau == 1) {
+#pragma unroll
+                for (int m = 0; m < 3; ++m) {
+                    const int32_t s3 = y[0][m] + y[1][m] + y[2][m];   // rows 3..5
+                    A0[m] += s3;
+                    A1[m] += s3;
+                    A2[m] = y[1][m] + y[2][m];                        // rows 4,5 of window 4..9
+                }
+            } else {
+#pragma unroll
+                for (int m = 0; m < 3; ++m) {
+                    const int32_t s2 = y[0][m] + y[1][m];             // rows 6,7
+                    A1[m] += s2;
+                    A2[m] += s2 + y[2][m];
+                    A3[m] = s2 + y[2][m];                             // rows 6..8 of window 6..11
+                }
+            }
+            if (++tau == 3) tau = 0;
+        }
+        emit(b1 - 1, Hr9, Hr911);   // the unit's last band, completed by the halo rows
+
+        if (kChecksum) {
+#pragma unroll
+            for (int off = 16; off > 0; off >>= 1) csacc += __shfl_xor_sync(0xffffffffu, csacc, off);
+            if (lane == 0 && csacc != 0)
+                atomicAdd(reinterpret_cast<unsigned long long*>(a.cs + plane / a.channels),
+                          static_cast<unsigned long long>(csacc));
+        }
+    }
+    if (tid == 0) ptx::bulk_wait<0>();
+}
+
+// -------------------------------------------------------------------------
+// Generic fused kernel: any W % 8 == 0, H % 9 == 0, int32 or uint8 input.
+// One thread per (plane, band, output column): recomputes the 12 Y values it
+// needs straight from global memory (L1/L2 absorb the overlap).  Correct for
+// every shape; used when the TMA kernel's geometry constraints do not hold.
+template <typename Tin, bool kChecksum>
+__global__ void __launch_bounds__(256)
+    fused_generic_kernel(const Tin* __restrict__ X, int32_t* __restrict__ Z, uint64_t* __restrict__ cs,
+                         int64_t planes, int32_t H, int32_t W, int32_t Ho, int32_t Wo, int32_t channels) {
+    const int32_t nb = H / 9;
+    const int64_t total = planes * nb * int64_t(Wo);
+    const int64_t stride = int64_t(gridDim.x) * blockDim.x;
+    const int64_t start = int64_t(blockIdx.x) * blockDim.x + threadIdx.x;
+    // warp-uniform trip count so the warp-level checksum reduction is safe
+    const int64_t warp_base = start - (threadIdx.x & 31);
+    for (int64_t base = warp_base; base < total; base += stride) {
+        const int64_t idx = base + (threadIdx.x & 31);
+        const bool live = idx < total;
+        uint64_t contrib = 0;
+        int64_t frame = -1;
+        if (live) {
+            const int32_t xo = int32_t(idx % Wo);
+            const int64_t rest = idx / Wo;
+            const int32_t b = int32_t(rest % nb);
+            const int64_t plane = rest / nb;
+            const int32_t rep = xo / 3, k = xo % 3;
+            const int32_t s0 = (k == 0) ? 0 : (k == 1 ? 2 : 5);
+            int32_t col[6];
+#pragma unroll
+            for (int t = 0; t < 6; ++t) {
+                int32_t c = 8 * rep + s0 + t;
+                col[t] = c >= W ? c - W : c;
+            }
+            const Tin* Xp = X + size_t(plane) * H * W;
+            int32_t yv[12];
+#pragma unroll
+            for (int j = 0; j < 12; ++j) {
+                int32_t row = 9 * b + j;
+                if (row >= H) row -= H;
+                const Tin* xr = Xp + size_t(row) * W;
+                int32_t S = 0;
+#pragma unroll
+                for (int t = 0; t < 6; ++t) S += int32_t(xr[col[t]]);
+                yv[j] = task_T(S);
+            }
+            int32_t* Zp = Z + size_t(plane) * Ho * Wo;
+            const int32_t chan = int32_t(plane % channels);
+#pragma unroll
+            for (int kk = 0; kk < 4; ++kk) {
+                int32_t S = 0;
+#pragma unroll
+                for (int t = 0; t < 6; ++t) S += yv[2 * kk + t];
+                const int32_t z = task_T(S);
+                const int32_t yo = 4 * b + kk;
+                Zp[size_t(yo) * Wo + xo] = z;
+                if (kChecksum)
+                    contrib += uint64_t(uint32_t(z)) * (1u + (uint64_t(chan) * Ho + yo) * uint64_t(Wo) + xo);
+            }
+            frame = plane / channels;
+        }
+        if (kChecksum) {
+            const int64_t f0 = __shfl_sync(0xffffffffu, frame, 0);
+            const bool uniform = __all_sync(0xffffffffu, frame == f0 || frame < 0);
+            if (uniform) {
+#pragma unroll
+                for (int off = 16; off > 0; off >>= 1) contrib += __shfl_xor_sync(0xffffffffu, contrib, off);
+                if ((threadIdx.x & 31) == 0 && f0 >= 0)
+                    atomicAdd(reinterpret_cast<unsigned long long*>(cs + f0), (unsigned long long)contrib);
+            } else if (live) {
+                atomicAdd(reinterpret_cast<unsigned long long*>(cs + frame), (unsigned long long)contrib);
+            }
+        }
+    }
+}
+
+using KernelFn = void (*)(const CUtensorMap, const FusedArgs);
+
+// Explicit instantiations live in fused_k_*.cu (compiled in parallel); these pick one.
+KernelFn tma_kernel_i32(bool checksum, int block, int cps);
+KernelFn tma_kernel_u8(bool checksum, int block, int cps);
+
+template <typename Tin, bool kChecksum>
+KernelFn pick_tma_kernel(int block, int cps) {
+    if (block <= 128 && cps >= 3) return fused_tma_kernel<Tin, kChecksum, 128, 4>;
+    if (block <= 320 && cps >= 2) return fused_tma_kernel<Tin, kChecksum, 320, 2>;
+    if (block <= 512) return fused_tma_kernel<Tin, kChecksum, 512, 1>;
+    return fused_tma_kernel<Tin, kChecksum, 1024, 1>;
+}
+
+}  // namespace fused
+}  // namespace aol

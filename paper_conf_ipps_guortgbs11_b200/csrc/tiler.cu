@@ -4,13 +4,16 @@
 //   gather : tiles[r][i]  = array[(o + P.r + F.i) mod s]     (Section IV, Fig. 4)
 //   scatter: array[(o + P.r + F.i) mod s] = tiles[r][i]      (Fig. 6, modarray P:L479)
 //
-// The host reduces o, P and F modulo the array extents once (so every partial
-// sum is non-negative) and validates that no sum can overflow int64.  Each
-// thread handles a run of kRun consecutive tile elements: it decomposes the
-// run's first flat index once, then walks the innermost pattern dimension
-// with an incremental (add, conditional subtract) update of every array
-// coordinate -- the tiler analogue of Fig. 11's inner `tl[0]` loop, without a
-// modulo per element.  Tile-side accesses are contiguous per thread.
+// The host reduces o, P and F modulo the array extents (every partial sum is
+// then non-negative) and classifies each array dimension: if no (r, i) can
+// push its coordinate past the extent, the `mod` is the identity there.  When
+// that holds for every dimension the tiler is an affine map of the flat tile
+// index -- offset = base + sum_d lin[d] * idx[d] -- and the LINEAR kernels
+// apply: one fast 32-bit division chain per thread and, when the innermost
+// pattern dimension walks contiguous memory, 16-byte vector accesses on both
+// sides.  Otherwise the GENERAL kernels evaluate the modulo per wrapping
+// dimension.  Tile-side accesses are always coalesced (consecutive threads,
+// consecutive tile elements).
 #include <cuda_runtime.h>
 
 #include <algorithm>
@@ -21,8 +24,6 @@
 namespace aol {
 
 namespace {
-
-constexpr int kRun = 8;
 
 template <int ES>
 struct Elem;
@@ -43,138 +44,159 @@ struct Elem<8> {
     using T = unsigned long long;
 };
 
-struct Walker {
-    int64_t idx[2 * AOL_MAX_RANK];
-    int64_t c[AOL_MAX_RANK];
-
-    __device__ __forceinline__ void seek(const TilerDev& td, int64_t g) {
-        for (int d = td.nd - 1; d >= 0; --d) {
-            const int64_t e = td.ext[d];
-            const int64_t q = g / e;
-            idx[d] = g - q * e;
-            g = q;
-        }
-        recompute(td);
-    }
-    __device__ __forceinline__ void recompute(const TilerDev& td) {
-        for (int a = 0; a < td.ra; ++a) {
-            int64_t v = td.org[a];
-            for (int d = 0; d < td.nd; ++d) v += td.coef[a][d] * idx[d];
-            c[a] = v % td.ashape[a];  // all terms non-negative: plain modulo == Euclidean
-        }
-    }
-    __device__ __forceinline__ int64_t offset(const TilerDev& td) const {
-        int64_t off = 0;
-        for (int a = 0; a < td.ra; ++a) off += c[a] * td.astride[a];
-        return off;
-    }
-    __device__ __forceinline__ void advance(const TilerDev& td) {
-        if (td.nd == 0) return;
-        const int last = td.nd - 1;
-        if (++idx[last] < td.ext[last]) {
-            for (int a = 0; a < td.ra; ++a) {
-                int64_t v = c[a] + td.coef[a][last];
-                if (v >= td.ashape[a]) v -= td.ashape[a];
-                c[a] = v;
-            }
-            return;
-        }
-        idx[last] = 0;
-        int d = last - 1;
-        while (d >= 0 && ++idx[d] == td.ext[d]) {
-            idx[d] = 0;
-            --d;
-        }
-        recompute(td);
-    }
+template <int BYTES>
+struct Vec;
+template <>
+struct Vec<1> {
+    using T = uint8_t;
+};
+template <>
+struct Vec<2> {
+    using T = uint16_t;
+};
+template <>
+struct Vec<4> {
+    using T = uint32_t;
+};
+template <>
+struct Vec<8> {
+    using T = uint2;
+};
+template <>
+struct Vec<16> {
+    using T = uint4;
 };
 
-template <int ES>
-__global__ void __launch_bounds__(256) gather_kernel(const TilerDev td, const void* __restrict__ array,
-                                                     void* __restrict__ tiles) {
-    using T = typename Elem<ES>::T;
-    const T* A = static_cast<const T*>(array);
-    T* G = static_cast<T*>(tiles);
-    const int64_t nruns = (td.total + kRun - 1) / kRun;
-    for (int64_t run = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; run < nruns;
-         run += int64_t(gridDim.x) * blockDim.x) {
-        const int64_t g0 = run * kRun;
-        const int n = (td.total - g0 < kRun) ? int(td.total - g0) : kRun;
-        Walker w;
-        w.seek(td, g0);
-        T v[kRun];
+constexpr int kND = 2 * AOL_MAX_RANK;
+
+// Decompose flat tile index g into the combined (rep ++ pattern) multi-index, last dim fastest.
+template <bool kFast32>
+__device__ __forceinline__ void decompose(const TilerDev& td, int64_t g, int64_t (&idx)[kND]) {
 #pragma unroll
-        for (int k = 0; k < kRun; ++k) {
-            if (k < n) {
-                v[k] = A[w.offset(td)];
-                if (k + 1 < n) w.advance(td);
+    for (int d = kND - 1; d >= 0; --d) {
+        if (d < td.nd) {
+            if (kFast32) {
+                const uint32_t n = uint32_t(g);
+                const uint32_t q = (__umulhi(n, td.fd_mul[d]) + n) >> td.fd_shift[d];
+                idx[d] = int64_t(n - q * uint32_t(td.ext[d]));
+                g = q;
+            } else {
+                const int64_t q = g / td.ext[d];
+                idx[d] = g - q * td.ext[d];
+                g = q;
             }
+        } else {
+            idx[d] = 0;
         }
-#pragma unroll
-        for (int k = 0; k < kRun; ++k)
-            if (k < n) G[g0 + k] = v[k];
     }
 }
 
-// mode 0: FAST (injective, plain stores); mode 1: SEQUENTIAL pass 1 (claim: max
-// flat index + 1 per target); mode 2: SEQUENTIAL pass 2 (write if we are the claim).
+__device__ __forceinline__ int64_t linear_offset(const TilerDev& td, const int64_t (&idx)[kND]) {
+    int64_t off = td.base;
+#pragma unroll
+    for (int d = 0; d < kND; ++d)
+        if (d < td.nd) off += td.lin[d] * idx[d];
+    return off;
+}
+
+__device__ __forceinline__ int64_t general_offset(const TilerDev& td, const int64_t (&idx)[kND]) {
+    int64_t off = 0;
+#pragma unroll
+    for (int a = 0; a < AOL_MAX_RANK; ++a) {
+        if (a < td.ra) {
+            int64_t v = td.org[a];
+#pragma unroll
+            for (int d = 0; d < kND; ++d)
+                if (d < td.nd) v += td.coef[a][d] * idx[d];
+            if (!((td.nowrap_mask >> a) & 1)) v %= td.ashape[a];   // all terms >= 0: % == Euclidean mod
+            off += v * td.astride[a];
+        }
+    }
+    return off;
+}
+
+// mode 0: gather; 1: FAST scatter; 2: SEQUENTIAL claim (max flat index + 1 per target);
+// 3: SEQUENTIAL write (store iff this element holds the claim).
+template <int ES, int V, bool kFast32, bool kLinear, int MODE>
+__global__ void __launch_bounds__(256) tiler_kernel(const TilerDev td, const void* __restrict__ src,
+                                                    void* __restrict__ dst, unsigned long long* __restrict__ ws) {
+    using T = typename Elem<ES>::T;
+    using VT = typename Vec<ES * V>::T;
+    const int64_t nvec = td.total / V;
+    for (int64_t v = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; v < nvec; v += int64_t(gridDim.x) * blockDim.x) {
+        const int64_t g = v * V;
+        int64_t idx[kND];
+        decompose<kFast32>(td, g, idx);
+        const int64_t off = kLinear ? linear_offset(td, idx) : general_offset(td, idx);
+        if (MODE == 0) {
+            // tiles[g .. g+V) = array[off .. off+V)   (V > 1 only when contiguous and aligned)
+            reinterpret_cast<VT*>(dst)[v] = reinterpret_cast<const VT*>(static_cast<const T*>(src) + off)[0];
+        } else if (MODE == 1) {
+            reinterpret_cast<VT*>(static_cast<T*>(dst) + off)[0] = reinterpret_cast<const VT*>(src)[v];
+        } else if (MODE == 2) {
+            atomicMax(ws + off, (unsigned long long)g + 1ull);
+        } else {
+            if (ws[off] == (unsigned long long)g + 1ull) static_cast<T*>(dst)[off] = static_cast<const T*>(src)[g];
+        }
+    }
+}
+
+int grid_for(int64_t n, int num_sms) {
+    return int(std::max<int64_t>(1, std::min<int64_t>((n + 255) / 256, int64_t(num_sms) * 32)));
+}
+
+template <int ES, int V, int MODE>
+aol_status_t launch_v(const TilerDev& td, const void* src, void* dst, unsigned long long* ws, int grid,
+                      cudaStream_t s) {
+    const bool fast = td.fast32 != 0, lin = td.linear != 0;
+    if (fast && lin)
+        tiler_kernel<ES, V, true, true, MODE><<<grid, 256, 0, s>>>(td, src, dst, ws);
+    else if (fast)
+        tiler_kernel<ES, V, true, false, MODE><<<grid, 256, 0, s>>>(td, src, dst, ws);
+    else if (lin)
+        tiler_kernel<ES, V, false, true, MODE><<<grid, 256, 0, s>>>(td, src, dst, ws);
+    else
+        tiler_kernel<ES, V, false, false, MODE><<<grid, 256, 0, s>>>(td, src, dst, ws);
+    AOL_LAUNCH_CHECK("tiler_kernel");
+    return AOL_OK;
+}
+
 template <int ES, int MODE>
-__global__ void __launch_bounds__(256) scatter_kernel(const TilerDev td, const void* __restrict__ tiles,
-                                                      void* __restrict__ array, unsigned long long* __restrict__ ws) {
-    using T = typename Elem<ES>::T;
-    const T* G = static_cast<const T*>(tiles);
-    T* A = static_cast<T*>(array);
-    const int64_t nruns = (td.total + kRun - 1) / kRun;
-    for (int64_t run = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; run < nruns;
-         run += int64_t(gridDim.x) * blockDim.x) {
-        const int64_t g0 = run * kRun;
-        const int n = (td.total - g0 < kRun) ? int(td.total - g0) : kRun;
-        Walker w;
-        w.seek(td, g0);
-#pragma unroll
-        for (int k = 0; k < kRun; ++k) {
-            if (k < n) {
-                const int64_t off = w.offset(td);
-                const unsigned long long tag = (unsigned long long)(g0 + k) + 1ull;
-                if (MODE == 0) {
-                    A[off] = G[g0 + k];
-                } else if (MODE == 1) {
-                    atomicMax(ws + off, tag);
-                } else {
-                    if (ws[off] == tag) A[off] = G[g0 + k];
-                }
-                if (k + 1 < n) w.advance(td);
-            }
-        }
+aol_status_t launch_es(const TilerDev& td, int vec, const void* src, void* dst, unsigned long long* ws,
+                       int num_sms, cudaStream_t s) {
+    const int grid = grid_for(td.total / vec, num_sms);
+    // vector width in elements: 16 / ES when the host proved contiguity + alignment, else 1
+    if (vec > 1 && ES * vec == 16) {
+        if constexpr (ES == 1) return launch_v<1, 16, MODE>(td, src, dst, ws, grid, s);
+        if constexpr (ES == 2) return launch_v<2, 8, MODE>(td, src, dst, ws, grid, s);
+        if constexpr (ES == 4) return launch_v<4, 4, MODE>(td, src, dst, ws, grid, s);
+        if constexpr (ES == 8) return launch_v<8, 2, MODE>(td, src, dst, ws, grid, s);
     }
+    return launch_v<ES, 1, MODE>(td, src, dst, ws, grid_for(td.total, num_sms), s);
 }
 
-int grid_for(int64_t total, int num_sms) {
-    const int64_t runs = (total + kRun - 1) / kRun;
-    return int(std::max<int64_t>(1, std::min<int64_t>((runs + 255) / 256, int64_t(num_sms) * 16)));
-}
-
-template <int ES>
-aol_status_t gather_es(const TilerDev& td, const void* a, void* t, int grid, cudaStream_t s) {
-    gather_kernel<ES><<<grid, 256, 0, s>>>(td, a, t);
-    AOL_LAUNCH_CHECK("gather_kernel");
-    return AOL_OK;
-}
-
-template <int ES>
-aol_status_t scatter_es(const TilerDev& td, const void* t, void* a, int seq, void* ws, int grid, cudaStream_t s) {
-    auto* w = static_cast<unsigned long long*>(ws);
-    if (!seq) {
-        scatter_kernel<ES, 0><<<grid, 256, 0, s>>>(td, t, a, w);
-        AOL_LAUNCH_CHECK("scatter_kernel");
-        return AOL_OK;
+template <int MODE>
+aol_status_t launch_mode(const TilerDev& td, int elsize, int vec, const void* src, void* dst,
+                         unsigned long long* ws, int num_sms, cudaStream_t s) {
+    switch (elsize) {
+        case 1: return launch_es<1, MODE>(td, vec, src, dst, ws, num_sms, s);
+        case 2: return launch_es<2, MODE>(td, vec, src, dst, ws, num_sms, s);
+        case 4: return launch_es<4, MODE>(td, vec, src, dst, ws, num_sms, s);
+        case 8: return launch_es<8, MODE>(td, vec, src, dst, ws, num_sms, s);
     }
-    AOL_CUDA_TRY(cudaMemsetAsync(ws, 0, size_t(td.array_elems) * 8, s));
-    scatter_kernel<ES, 1><<<grid, 256, 0, s>>>(td, t, a, w);
-    AOL_LAUNCH_CHECK("scatter_kernel(claim)");
-    scatter_kernel<ES, 2><<<grid, 256, 0, s>>>(td, t, a, w);
-    AOL_LAUNCH_CHECK("scatter_kernel(write)");
-    return AOL_OK;
+    return fail(AOL_E_DTYPE, "element size must be 1, 2, 4 or 8 bytes");
+}
+
+// Largest usable vector (elements): contiguous innermost dim, divisibility and alignment.
+int vector_width(const TilerDev& td, int elsize, const void* p_array, const void* p_tiles) {
+    const int v = 16 / elsize;
+    if (!td.linear || td.nd == 0 || v <= 1) return 1;
+    const int last = td.nd - 1;
+    if (td.lin[last] != 1 || td.ext[last] % v != 0 || td.base % v != 0) return 1;
+    for (int d = 0; d < last; ++d)
+        if (td.lin[d] % v != 0) return 1;
+    if ((reinterpret_cast<uintptr_t>(p_array) | reinterpret_cast<uintptr_t>(p_tiles)) % 16) return 1;
+    return v;
 }
 
 }  // namespace
@@ -184,14 +206,8 @@ aol_status_t launch_gather(const TilerDev& td, int elsize, const void* d_array, 
     DeviceInfo dev;
     aol_status_t st = device_info(&dev);
     if (st != AOL_OK) return st;
-    const int grid = grid_for(td.total, dev.num_sms);
-    switch (elsize) {
-        case 1: return gather_es<1>(td, d_array, d_tiles, grid, s);
-        case 2: return gather_es<2>(td, d_array, d_tiles, grid, s);
-        case 4: return gather_es<4>(td, d_array, d_tiles, grid, s);
-        case 8: return gather_es<8>(td, d_array, d_tiles, grid, s);
-    }
-    return fail(AOL_E_DTYPE, "element size must be 1, 2, 4 or 8 bytes");
+    return launch_mode<0>(td, elsize, vector_width(td, elsize, d_array, d_tiles), d_array, d_tiles, nullptr,
+                          dev.num_sms, s);
 }
 
 aol_status_t launch_scatter(const TilerDev& td, int elsize, const void* d_tiles, void* d_array, int sequential,
@@ -200,14 +216,14 @@ aol_status_t launch_scatter(const TilerDev& td, int elsize, const void* d_tiles,
     DeviceInfo dev;
     aol_status_t st = device_info(&dev);
     if (st != AOL_OK) return st;
-    const int grid = grid_for(td.total, dev.num_sms);
-    switch (elsize) {
-        case 1: return scatter_es<1>(td, d_tiles, d_array, sequential, d_ws, grid, s);
-        case 2: return scatter_es<2>(td, d_tiles, d_array, sequential, d_ws, grid, s);
-        case 4: return scatter_es<4>(td, d_tiles, d_array, sequential, d_ws, grid, s);
-        case 8: return scatter_es<8>(td, d_tiles, d_array, sequential, d_ws, grid, s);
-    }
-    return fail(AOL_E_DTYPE, "element size must be 1, 2, 4 or 8 bytes");
+    auto* ws = static_cast<unsigned long long*>(d_ws);
+    if (!sequential)
+        return launch_mode<1>(td, elsize, vector_width(td, elsize, d_array, d_tiles), d_tiles, d_array, nullptr,
+                              dev.num_sms, s);
+    AOL_CUDA_TRY(cudaMemsetAsync(d_ws, 0, size_t(td.array_elems) * 8, s));
+    st = launch_mode<2>(td, elsize, 1, d_tiles, d_array, ws, dev.num_sms, s);
+    if (st != AOL_OK) return st;
+    return launch_mode<3>(td, elsize, 1, d_tiles, d_array, ws, dev.num_sms, s);
 }
 
 }  // namespace aol

@@ -165,3 +165,14 @@ def test_package_has_no_oracle_dependency():
                 with open(os.path.join(dirpath, fn)) as f:
                     src = f.read()
                 assert "import oracle" not in src and "from oracle" not in src and "aol_oracle" not in src, fn
+
+
+def test_kernel_division_identities():
+    """The kernels rewrite Fig. 5's tmp/6 - tmp%6 (C semantics) as 7*(tmp/6) - tmp, and for
+    non-negative 8-bit sums use tmp/6 == (tmp*43691) >> 18 (32-bit).  Both are checked
+    exhaustively on their domains here (numpy trunc/fmod = C99 truncating / and %)."""
+    S = np.arange(-(1 << 20), 1 << 20, dtype=np.int64)
+    q = np.trunc(S / 6).astype(np.int64)
+    assert np.array_equal(q - np.fmod(S, 6), 7 * q - S)
+    U = np.arange(0, 98304, dtype=np.uint64)
+    assert np.array_equal(((U * np.uint64(43691)) & np.uint64(0xFFFFFFFF)) >> np.uint64(18), U // np.uint64(6))

@@ -79,7 +79,7 @@ def test_fused_vs_oracle(orc, shape, kernel):
 @pytest.mark.parametrize("opts", [
     {"bands_per_unit": 1}, {"bands_per_unit": 2}, {"bands_per_unit": 7}, {"bands_per_unit": 40},
     {"stages": 2}, {"stages": 3, "bands_per_unit": 5}, {"ctas_per_sm": 2}, {"ctas_per_sm": 2, "stages": 2},
-    {"flags": 1}, {"flags": 1, "bands_per_unit": 1, "stages": 2},
+    {"flags": 1}, {"flags": 1, "bands_per_unit": 1, "stages": 2}, {"ctas_per_sm": 4}, {"ctas_per_sm": 8, "stages": 2},
 ])
 def test_fused_launch_options(orc, opts):
     """Unit boundaries, ring wrap-around and CTA residency do not change results."""
@@ -111,15 +111,36 @@ def test_generic_only_shapes(orc, shape):
         aol.downscale_frame(torch.from_numpy(xh).cuda(), opts={"kernel": 1})
 
 
-def test_fused_u8_input(orc):
-    """8-bit samples give the same integers, hence the same outputs."""
-    xh = synth.frames(21, 0, 2, 3, 36, 128, "uniform")
+@pytest.mark.parametrize("shape,kernel", [
+    ((2, 3, 36, 128), 1), ((1, 3, 1080, 1920), 1), ((3, 3, 288, 352), 1), ((1, 1, 9, 16), 1),
+    ((2, 2, 27, 3840), 1), ((1, 2, 18, 40), 2), ((2, 3, 36, 128), 2),
+])
+@pytest.mark.parametrize("kind", ["uniform", "dark", "ramp"])
+def test_fused_u8_input(orc, shape, kernel, kind):
+    """8-bit samples give the same integers, hence the same outputs (NEXT row f1)."""
+    N, C, H, W = shape
+    if kind == "ramp" and W > 256:
+        kind = "uniform"
+    xh = synth.frames(21, 0, N, C, H, W, kind)
     zo, cso = run_oracle(orc, xh)
     x8 = torch.from_numpy(xh.astype(np.uint8)).cuda()
-    z, cs = aol.downscale_frame(x8, checksums=True)
+    plan = aol.downscale_frame_plan(N, C, H, W, dtype=torch.uint8, opts={"kernel": kernel})
+    assert plan["kernel"] == kernel
+    z, cs = aol.downscale_frame(x8, checksums=True, opts={"kernel": kernel})
     torch.cuda.synchronize()
     assert np.array_equal(z.cpu().numpy(), zo)
     assert np.array_equal(np_u64(cs), cso)
+
+
+def test_fused_u8_launch_options(orc):
+    xh = synth.frames(22, 0, 3, 3, 117, 512, "uniform")
+    zo, cso = run_oracle(orc, xh)
+    x8 = torch.from_numpy(xh.astype(np.uint8)).cuda()
+    for o in ({"bands_per_unit": 1}, {"stages": 2}, {"ctas_per_sm": 2}, {"ctas_per_sm": 4}, {"flags": 1}):
+        z, cs = aol.downscale_frame(x8, checksums=True, opts=dict(o, kernel=1))
+        torch.cuda.synchronize()
+        assert np.array_equal(z.cpu().numpy(), zo), o
+        assert np.array_equal(np_u64(cs), cso), o
 
 
 def test_no_checksum_and_zero_frames(orc):
@@ -188,6 +209,39 @@ def test_tiler_gather_scatter_vs_oracle(orc, seed):
         aol.tiler_scatter(gt, torch.from_numpy(Gs).cuda().reshape(G.shape), arr2, mode="fast")
         torch.cuda.synchronize()
         assert np.array_equal(arr2.cpu().numpy(), So)
+
+
+LINEAR_TILERS = [
+    # (array, rep, pattern, origin, paving, fitting): no coordinate wraps -> affine offsets
+    ([64, 96], [8, 12], [8, 8], [0, 0], [[8, 0], [0, 8]], [[1, 0], [0, 1]]),           # 8x8 blocks (vector path)
+    ([4, 32, 64], [4, 4, 8], [8, 8], [0, 0, 0], [[1, 0, 0], [0, 8, 0], [0, 0, 8]], [[0, 0], [1, 0], [0, 1]]),
+    ([50, 40], [6, 5], [3, 7], [2, 1], [[8, 0], [0, 8]], [[1, 0], [0, 1]]),             # offset, odd pattern
+    ([37, 23], [23], [37], [0, 0], [[0], [1]], [[1], [0]]),                            # transpose column gather
+    ([128], [15], [16], [0], [[8]], [[1]]),                                           # overlapping windows
+]
+
+
+@pytest.mark.parametrize("case", range(len(LINEAR_TILERS)))
+@pytest.mark.parametrize("dtype", [np.uint8, np.int16, np.int32, np.int64])
+def test_tiler_linear_paths(orc, case, dtype):
+    """Affine (non-wrapping) tilers take the linear kernels, incl. 16-byte vector accesses."""
+    arr, rep, pat, o, P, F = LINEAR_TILERS[case]
+    rng = np.random.default_rng(case)
+    A = np.asarray(rng.integers(0, 100, size=arr)).astype(dtype)
+    ot = orc.make_tiler(arr, rep, pat, o, P, F)
+    gt = aol.make_tiler(arr, rep, pat, o, P, F)
+    Go = orc.gather(ot, A)
+    G = aol.tiler_gather(gt, torch.from_numpy(A).cuda())
+    torch.cuda.synchronize()
+    assert np.array_equal(G.cpu().numpy(), Go)
+    Gs = np.asarray(rng.integers(0, 100, size=Go.shape)).astype(dtype)
+    bg = np.asarray(rng.integers(0, 100, size=A.shape)).astype(dtype)
+    So = orc.scatter(ot, Gs, bg)
+    for mode in (["fast", "sequential"] if aol.tiler_is_injective(gt) else ["sequential"]):
+        arr_t = torch.from_numpy(bg.copy()).cuda()
+        aol.tiler_scatter(gt, torch.from_numpy(Gs).cuda(), arr_t, mode=mode)
+        torch.cuda.synchronize()
+        assert np.array_equal(arr_t.cpu().numpy(), So), mode
 
 
 def test_tiler_paper_presets_on_gpu(orc):

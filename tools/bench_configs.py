@@ -1,0 +1,151 @@
+#!/usr/bin/env python
+"""Secondary measurements for every BASELINE.json config (bench.py times configs[1] only).
+
+One JSON line per measurement (CUDA events on the launching stream, median of N,
+after warm-up).  Algorithmic bytes: each input element read once, each output
+element written once.
+
+  d1   single HD frame, latency (warm L2 and cold L2 = 512 MB flush before each launch)
+  d2x  300 HD frames: fused TMA kernel vs generic fused kernel vs unfused H -> V -> checksum
+  d3   generic tiler perf instance: array {64,1024,1024} i32, rep {64,128,128}, pattern {8,8}
+  d4   64 frames of 3840x2160 (4K), same ratios
+  f1   300 HD frames with uint8 samples
+  f4   CIF 352x288, 2000 frames (Section III)
+"""
+import argparse
+import json
+import os
+import statistics
+import sys
+
+import torch
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+sys.path.insert(0, ROOT)
+import paper_conf_ipps_guortgbs11_b200 as aol  # noqa: E402
+
+
+def timed(fn, reps=20, warm=3, before=None):
+    s = torch.cuda.current_stream()
+    for _ in range(warm):
+        if before:
+            before()
+        fn()
+    torch.cuda.synchronize()
+    ts = []
+    for _ in range(reps):
+        if before:
+            before()
+        a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        a.record(s)
+        fn()
+        b.record(s)
+        torch.cuda.synchronize()
+        ts.append(a.elapsed_time(b))
+    return statistics.median(ts), min(ts)
+
+
+def peak():
+    try:
+        return float(json.load(open(os.path.join(ROOT, "MEASURED_PEAKS.json")))["hbm_gbs"])
+    except Exception:
+        return 6650.0
+
+
+def emit(d):
+    print(json.dumps(d), flush=True)
+
+
+def frames_bytes(N, C, H, W, es=4):
+    return N * C * (H * W * es + (4 * (H // 9)) * (3 * (W // 8)) * 4)
+
+
+def fused_line(name, N, C, H, W, dtype=torch.int32, opts=None, reps=20):
+    x = aol.synth_frames(3, 0, N, C, H, W, "uniform", dtype=dtype)
+    z = torch.empty((N, C, 4 * (H // 9), 3 * (W // 8)), dtype=torch.int32, device="cuda")
+    cs = torch.empty(N, dtype=torch.uint64, device="cuda")
+    med, mn = timed(lambda: aol.downscale_frame(x, out=z, checksums=cs, opts=opts), reps=reps)
+    b = frames_bytes(N, C, H, W, x.element_size())
+    plan = aol.downscale_frame_plan(N, C, H, W, dtype=dtype, opts=opts)
+    emit({"config": name, "shape": [N, C, H, W], "dtype": str(dtype).split(".")[-1], "ms": med, "min_ms": mn,
+          "frames_per_s": N / (med / 1e3), "GBps": b / (med / 1e3) / 1e9, "frac": b / (med / 1e3) / 1e9 / peak(),
+          "kernel": plan["kernel"], "plan": plan})
+    del x, z, cs
+    torch.cuda.empty_cache()
+
+
+def main():
+    p = argparse.ArgumentParser()
+    p.add_argument("--only", default="")
+    a = p.parse_args()
+    only = set(a.only.split(",")) if a.only else None
+
+    def want(k):
+        return only is None or k in only
+
+    torch.cuda.set_device(0)
+    if want("d1"):
+        N, C, H, W = 1, 3, 1080, 1920
+        x = aol.synth_frames(0, 0, N, C, H, W)
+        z = torch.empty((N, C, 480, 720), dtype=torch.int32, device="cuda")
+        cs = torch.empty(N, dtype=torch.uint64, device="cuda")
+        flush = torch.empty(512 << 20, dtype=torch.uint8, device="cuda")
+        warm, _ = timed(lambda: aol.downscale_frame(x, out=z, checksums=cs), reps=50)
+        cold, _ = timed(lambda: aol.downscale_frame(x, out=z, checksums=cs), reps=50, before=lambda: flush.fill_(1))
+        b = frames_bytes(N, C, H, W)
+        emit({"config": "d1 single HD frame", "warm_l2_us": warm * 1e3, "cold_l2_us": cold * 1e3,
+              "roofline_floor_us": b / peak() / 1e3, "cold_GBps": b / (cold / 1e3) / 1e9,
+              "plan": aol.downscale_frame_plan(N, C, H, W)})
+        del flush
+    if want("d2x"):
+        N, C, H, W = 300, 3, 1080, 1920
+        fused_line("d2 fused TMA kernel", N, C, H, W)
+        fused_line("d2 generic fused kernel (kernel=2)", N, C, H, W, opts={"kernel": 2}, reps=5)
+        x = aol.synth_frames(0, 0, N, C, H, W)
+        y = torch.empty((N, C, H, 720), dtype=torch.int32, device="cuda")
+        z = torch.empty((N, C, 480, 720), dtype=torch.int32, device="cuda")
+        cs = torch.empty(N, dtype=torch.uint64, device="cuda")
+
+        def unfused():
+            aol.downscale_h(x, out=y)
+            aol.downscale_v(y, out=z)
+            aol.frame_checksum(z, out=cs)
+
+        med, _ = timed(unfused, reps=10)
+        th, _ = timed(lambda: aol.downscale_h(x, out=y), reps=10)
+        tv, _ = timed(lambda: aol.downscale_v(y, out=z), reps=10)
+        b = frames_bytes(N, C, H, W)
+        emit({"config": "d2 unfused H -> V -> checksum (Y through HBM)", "ms": med, "frames_per_s": N / (med / 1e3),
+              "GBps_algorithmic": b / (med / 1e3) / 1e9, "h_ms": th, "v_ms": tv,
+              "h_GBps": (x.numel() * 4 + y.numel() * 4) / (th / 1e3) / 1e9,
+              "v_GBps": (y.numel() * 4 + z.numel() * 4) / (tv / 1e3) / 1e9})
+        del x, y, z, cs
+        torch.cuda.empty_cache()
+    if want("d3"):
+        t = aol.make_tiler([64, 1024, 1024], [64, 128, 128], [8, 8], [0, 0, 0],
+                           [[1, 0, 0], [0, 8, 0], [0, 0, 8]], [[0, 0], [1, 0], [0, 1]])
+        A = torch.randint(0, 1 << 30, (64, 1024, 1024), dtype=torch.int32, device="cuda")
+        G = torch.empty((64, 128, 128, 8, 8), dtype=torch.int32, device="cuda")
+        tg, _ = timed(lambda: aol.tiler_gather(t, A, out=G))
+        B = torch.empty_like(A)
+        ts, _ = timed(lambda: aol.tiler_scatter(t, G, B, mode="fast"))
+        tq, _ = timed(lambda: aol.tiler_scatter(t, G, B, mode="sequential",
+                                                workspace=torch.empty(A.numel() * 8, dtype=torch.uint8,
+                                                                      device="cuda")), reps=5)
+        nb = 2 * A.numel() * 4
+        emit({"config": "d3 generic tiler {64,1024,1024} i32 -> 8x8 tiles", "gather_ms": tg,
+              "gather_GBps": nb / (tg / 1e3) / 1e9, "scatter_fast_ms": ts, "scatter_fast_GBps": nb / (ts / 1e3) / 1e9,
+              "scatter_seq_ms": tq, "gather_frac": nb / (tg / 1e3) / 1e9 / peak(),
+              "check_gather_is_blocking": bool(torch.equal(G[1, 2, 3], A[1, 16:24, 24:32]))})
+        del A, G, B
+        torch.cuda.empty_cache()
+    if want("d4"):
+        fused_line("d4 4K batch", 64, 3, 2160, 3840)
+    if want("f1"):
+        fused_line("f1 HD uint8 input", 300, 3, 1080, 1920, dtype=torch.uint8)
+    if want("f4"):
+        fused_line("f4 CIF 2000 frames", 2000, 3, 288, 352)
+
+
+if __name__ == "__main__":
+    main()
