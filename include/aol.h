@@ -226,6 +226,49 @@ AOL_API aol_status_t aol_downscale_frame_host(const void* h_in, aol_dtype_t in_d
                                       int64_t chunk_frames, void* d_workspace, size_t ws_bytes,
                                       cudaStream_t s_h2d, cudaStream_t s_compute, cudaStream_t s_d2h);
 
+/* ------------------------------------ generic fused repetition (NEXT row f3) */
+
+#define AOL_MAX_FILTER_PATTERN 64 /* input pattern elements */
+#define AOL_MAX_WINDOWS 16        /* output pattern elements */
+
+/* One ArrayOL repetition, fully described at run time: an input tiler, a
+ * windowed-sum task and an output tiler -- the SaC "generic" downscaler of
+ * Fig. 4 (input_tiler) + Fig. 5 (task) + Fig. 6 (generic_output_tiler),
+ * P:L384-471, generalised to any window layout:
+ *   for every repetition r (in.rep_shape == out.rep_shape):
+ *     p      = the in.pattern elements gathered at r (flattened row-major)
+ *     tile[k] = S/divisor - S%divisor,  S = sum_{t<window_len} p[window_start[k] + t]   (C int)
+ *     out[(o' + P'.r + F'.k) mod s'] = tile[k]          (k < n_windows = out pattern elements)
+ * The paper's filters are presets (aol_filter_preset).  Gather, task and
+ * scatter run in ONE kernel (no intermediate arrays: WLF for arbitrary
+ * tilers).  Array extents must be < 2^31; the output tiler must be injective
+ * (ArrayOL single assignment) or results at colliding cells are unspecified. */
+typedef struct {
+    aol_tiler_t in;
+    aol_tiler_t out;
+    int32_t n_windows;  /* 1..AOL_MAX_WINDOWS, = out pattern element count          */
+    int32_t window_len; /* >= 1; window_start[k] + window_len <= in pattern elements */
+    int32_t divisor;    /* != 0                                                       */
+    int32_t window_start[AOL_MAX_WINDOWS];
+} aol_filter_t;
+
+typedef enum {
+    AOL_FILTER_H = 0, /* horizontal filter of Fig. 10 + Fig. 5 on [planes][H][W]   -> [planes][H][3W/8]  */
+    AOL_FILTER_V = 1  /* vertical filter (reading Z1/Z2) on [planes][H][W]         -> [planes][4H/9][W]  */
+} aol_filter_kind_t;
+
+/* The paper's filters as 3-D repetitions over a stack of planes (the plane index is one more
+ * repetition dimension with paving 1 -- time/channels as array dimensions). */
+AOL_API aol_status_t aol_filter_preset(aol_filter_kind_t which, int64_t planes, int64_t H, int64_t W,
+                                       aol_filter_t* out);
+
+/* Check a filter description (ranks, shapes, windows, divisor, int32 ranges).  Host only. */
+AOL_API aol_status_t aol_filter_validate(const aol_filter_t* f);
+
+/* Apply a filter: d_in int32 shaped f->in.array_shape, d_out int32 shaped f->out.array_shape
+ * (cells no repetition writes keep their value).  4-byte aligned.  Async on s. */
+AOL_API aol_status_t aol_filter_apply(const aol_filter_t* f, const int32_t* d_in, int32_t* d_out, cudaStream_t s);
+
 /* ------------------------------------------- synthetic input (test support) */
 
 /* Fill d_out [nframes][channels][H][W] with the counter-based synthetic frames

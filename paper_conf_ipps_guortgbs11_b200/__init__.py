@@ -17,15 +17,16 @@ from typing import Optional, Sequence
 import torch
 
 from . import _lib
-from ._lib import (AolError, I16, I32, I64, PRESET_H_IN, PRESET_H_OUT, PRESET_V_IN, PRESET_V_OUT, RAW8, RAW16,
-                   RAW32, RAW64, SCATTER_FAST, SCATTER_SEQUENTIAL, U8, aol_launch_opts_t, aol_plan_t,
-                   aol_tiler_t, check, lib)
+from ._lib import (FILTER_H, FILTER_V, AolError, I16, I32, I64, PRESET_H_IN, PRESET_H_OUT, PRESET_V_IN,
+                   PRESET_V_OUT, RAW8, RAW16, RAW32, RAW64, SCATTER_FAST, SCATTER_SEQUENTIAL, U8, aol_filter_t,
+                   aol_launch_opts_t, aol_plan_t, aol_tiler_t, check, lib)
 
 __all__ = [
     "AolError", "version", "make_tiler", "tiler_preset", "tiler_validate", "tiler_is_injective",
     "tiler_gather", "tiler_scatter", "downscale_h", "downscale_v", "downscale_frame", "downscale_frame_plan",
     "frame_checksum", "downscale_frame_host", "synth_frames", "library_path",
     "PRESET_H_IN", "PRESET_H_OUT", "PRESET_V_IN", "PRESET_V_OUT", "SYNTH_KINDS",
+    "make_filter", "filter_preset", "filter_validate", "filter_apply", "FILTER_H", "FILTER_V",
 ]
 
 SYNTH_KINDS = {"uniform": 0, "dark": 1, "signed": 2, "ramp": 3, "constant": 4}
@@ -136,6 +137,43 @@ def tiler_scatter(t: aol_tiler_t, tiles: torch.Tensor, array: torch.Tensor, mode
     check(lib().aol_tiler_scatter(ctypes.byref(t), _dtype_code(array), _dev(tiles, "tiles"),
                                   _dev(array, "array"), m, ws_ptr, ws_bytes, _stream(stream)))
     return array
+
+
+# ------------------------------------------------- generic repetition (f3)
+
+def make_filter(tin: aol_tiler_t, tout: aol_tiler_t, window_start: Sequence[int], window_len: int,
+                divisor: int) -> aol_filter_t:
+    """A run-time ArrayOL repetition: gather with tin, windowed-sum task, scatter with tout."""
+    f = aol_filter_t()
+    f.in_, f.out = tin, tout
+    f.n_windows = len(window_start)
+    f.window_len, f.divisor = int(window_len), int(divisor)
+    for k, v in enumerate(window_start):
+        f.window_start[k] = int(v)
+    return f
+
+
+def filter_preset(kind: int, planes: int, H: int, W: int) -> aol_filter_t:
+    f = aol_filter_t()
+    check(lib().aol_filter_preset(kind, planes, H, W, ctypes.byref(f)))
+    return f
+
+
+def filter_validate(f: aol_filter_t) -> None:
+    check(lib().aol_filter_validate(ctypes.byref(f)))
+
+
+def filter_apply(f: aol_filter_t, x: torch.Tensor, out: Optional[torch.Tensor] = None,
+                 stream: Optional[torch.cuda.Stream] = None) -> torch.Tensor:
+    """Run the fused generic repetition: x int32 shaped f.in_ array -> out int32 shaped f.out array."""
+    a_in, _, _ = _shapes(f.in_)
+    a_out, _, _ = _shapes(f.out)
+    if x.dtype != torch.int32 or tuple(x.shape) != a_in:
+        raise ValueError(f"x must be int32 {a_in}")
+    if out is None:
+        out = torch.zeros(a_out, dtype=torch.int32, device=x.device)
+    check(lib().aol_filter_apply(ctypes.byref(f), _dev(x, "x"), _dev(out, "out"), _stream(stream)))
+    return out
 
 
 # ------------------------------------------------------------------ filters

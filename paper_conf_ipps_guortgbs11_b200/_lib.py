@@ -45,6 +45,16 @@ class aol_tiler_t(ctypes.Structure):
     ]
 
 
+MAX_FILTER_PATTERN, MAX_WINDOWS = 64, 16
+FILTER_H, FILTER_V = 0, 1
+
+
+class aol_filter_t(ctypes.Structure):
+    _fields_ = [("in_", aol_tiler_t), ("out", aol_tiler_t), ("n_windows", ctypes.c_int32),
+                ("window_len", ctypes.c_int32), ("divisor", ctypes.c_int32),
+                ("window_start", ctypes.c_int32 * MAX_WINDOWS)]
+
+
 class aol_launch_opts_t(ctypes.Structure):
     _fields_ = [("ctas_per_sm", ctypes.c_int32), ("stages", ctypes.c_int32),
                 ("bands_per_unit", ctypes.c_int32), ("kernel", ctypes.c_int32),
@@ -62,6 +72,7 @@ _I64 = ctypes.c_int64
 _I32 = ctypes.c_int32
 _ST = ctypes.c_int  # aol_status_t
 _TP = ctypes.POINTER(aol_tiler_t)
+_FP = ctypes.POINTER(aol_filter_t)
 
 SIGNATURES = {
     "aol_version": ([], ctypes.c_int),
@@ -83,6 +94,9 @@ SIGNATURES = {
     "aol_downscale_frame_host_workspace_bytes": ([ctypes.c_int, _I64, _I64, _I64, _I64], ctypes.c_size_t),
     "aol_downscale_frame_host": ([_P, ctypes.c_int, _P, _I64, _I64, _I64, _I64, _P, _I64, _P, ctypes.c_size_t,
                                   _P, _P, _P], _ST),
+    "aol_filter_preset": ([ctypes.c_int, _I64, _I64, _I64, _FP], _ST),
+    "aol_filter_validate": ([_FP], _ST),
+    "aol_filter_apply": ([_FP, _P, _P, _P], _ST),
     "aol_synth_frames": ([ctypes.c_uint64, _I64, _I64, _I64, _I64, _I64, _I32, _I32, ctypes.c_int, _P, _P], _ST),
 }
 

@@ -1,0 +1,287 @@
+// filter.cu -- NEXT row f3: one ArrayOL repetition (input tiler -> windowed-sum task -> output
+// tiler) described at RUN TIME and executed by one fused kernel.  This is the "generic"
+// formulation of the paper's SaC downscaler (Fig. 4 input_tiler, Fig. 5 task, Fig. 6
+// generic_output_tiler), whose GPU version lost 4.5x (H) / 3x (V) to the
+// non-generic one because the generic output tiler ran on the host.  Here all
+// three steps stay on the device in a single kernel, so the comparison with the specialised
+// K-5 measures what generality costs on B200 (tools/bench_configs.py, config f3).
+//
+// Per repetition r (one thread): base coordinates of both tilers are o' + P'.r reduced mod
+// the extents once; the pattern-element and output-element offsets F'.i are host-precomputed
+// tables already reduced mod the extents, so every element costs an add, a conditional
+// subtract and an FMA per array dimension.
+#include <cuda_runtime.h>
+
+#include <algorithm>
+#include <cstdint>
+#include <cstring>
+
+#include "common.h"
+
+namespace aol {
+
+namespace {
+
+struct FilterDev {
+    int32_t ra_in, ra_out, rr, n_in, n_win, len, divisor, fast32;
+    int64_t nrep;
+    int32_t rep_ext[AOL_MAX_RANK];
+    uint32_t fd_mul[AOL_MAX_RANK], fd_shift[AOL_MAX_RANK];
+    int32_t s_in[AOL_MAX_RANK], s_out[AOL_MAX_RANK];
+    int64_t st_in[AOL_MAX_RANK], st_out[AOL_MAX_RANK];
+    int32_t o_in[AOL_MAX_RANK], o_out[AOL_MAX_RANK];
+    int32_t P_in[AOL_MAX_RANK][AOL_MAX_RANK], P_out[AOL_MAX_RANK][AOL_MAX_RANK];
+    int32_t start[AOL_MAX_WINDOWS];
+    int32_t f_in[AOL_MAX_FILTER_PATTERN][AOL_MAX_RANK];  // F'.i(p) mod s, per input pattern element
+    int32_t f_out[AOL_MAX_WINDOWS][AOL_MAX_RANK];        // F'.i(k) mod s, per output element
+};
+
+template <bool kFast32>
+__global__ void __launch_bounds__(256) filter_kernel(const FilterDev fd, const int32_t* __restrict__ in,
+                                                     int32_t* __restrict__ out) {
+    for (int64_t r = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; r < fd.nrep;
+         r += int64_t(gridDim.x) * blockDim.x) {
+        // repetition multi-index (last dim fastest)
+        int64_t ridx[AOL_MAX_RANK];
+        int64_t g = r;
+#pragma unroll
+        for (int j = AOL_MAX_RANK - 1; j >= 0; --j) {
+            if (j < fd.rr) {
+                if (kFast32) {
+                    const uint32_t n = uint32_t(g);
+                    const uint32_t q = (__umulhi(n, fd.fd_mul[j]) + n) >> fd.fd_shift[j];
+                    ridx[j] = int64_t(n - q * uint32_t(fd.rep_ext[j]));
+                    g = q;
+                } else {
+                    const int64_t q = g / fd.rep_ext[j];
+                    ridx[j] = g - q * fd.rep_ext[j];
+                    g = q;
+                }
+            } else {
+                ridx[j] = 0;
+            }
+        }
+        // reference points o' + P'.r  (mod s), Section IV
+        int32_t bin[AOL_MAX_RANK], bout[AOL_MAX_RANK];
+#pragma unroll
+        for (int a = 0; a < AOL_MAX_RANK; ++a) {
+            int64_t vi = fd.o_in[a], vo = fd.o_out[a];
+#pragma unroll
+            for (int j = 0; j < AOL_MAX_RANK; ++j) {
+                if (j < fd.rr) {
+                    vi += int64_t(fd.P_in[a][j]) * ridx[j];
+                    vo += int64_t(fd.P_out[a][j]) * ridx[j];
+                }
+            }
+            bin[a] = a < fd.ra_in ? int32_t(vi % fd.s_in[a]) : 0;
+            bout[a] = a < fd.ra_out ? int32_t(vo % fd.s_out[a]) : 0;
+        }
+        for (int k = 0; k < fd.n_win; ++k) {
+            // task (Fig. 5): S over the window, tile = S/d - S%d
+            int32_t S = 0;
+            for (int t = 0; t < fd.len; ++t) {
+                const int p = fd.start[k] + t;
+                int64_t off = 0;
+#pragma unroll
+                for (int a = 0; a < AOL_MAX_RANK; ++a) {
+                    if (a < fd.ra_in) {
+                        int32_t c = bin[a] + fd.f_in[p][a];   // pattern element
+                        if (c >= fd.s_in[a]) c -= fd.s_in[a];
+                        off += int64_t(c) * fd.st_in[a];
+                    }
+                }
+                S += __ldg(in + off);
+            }
+            const int32_t tile = S / fd.divisor - S % fd.divisor;
+            int64_t off = 0;
+#pragma unroll
+            for (int a = 0; a < AOL_MAX_RANK; ++a) {
+                if (a < fd.ra_out) {
+                    int32_t c = bout[a] + fd.f_out[k][a];       // output tiler (Fig. 6)
+                    if (c >= fd.s_out[a]) c -= fd.s_out[a];
+                    off += int64_t(c) * fd.st_out[a];
+                }
+            }
+            out[off] = tile;
+        }
+    }
+}
+
+int64_t emod(int64_t a, int64_t m) {
+    const int64_t r = a % m;
+    return r < 0 ? r + m : r;
+}
+
+int64_t elems(const int64_t* s, int n) {
+    int64_t p = 1;
+    for (int k = 0; k < n; ++k) p *= s[k];
+    return p;
+}
+
+// pattern element p (flattened row-major) -> its multi-index
+void unflatten(int64_t p, const int64_t* shape, int n, int64_t* idx) {
+    for (int k = n - 1; k >= 0; --k) {
+        idx[k] = p % shape[k];
+        p /= shape[k];
+    }
+}
+
+aol_status_t check_filter(const aol_filter_t* f) {
+    if (!f) return fail(AOL_E_INVALID, "filter is NULL");
+    aol_status_t st = aol_tiler_validate(&f->in);
+    if (st != AOL_OK) return st;
+    st = aol_tiler_validate(&f->out);
+    if (st != AOL_OK) return st;
+    if (f->in.rep_rank != f->out.rep_rank) return fail(AOL_E_SHAPE, "input and output repetition spaces differ");
+    for (int j = 0; j < f->in.rep_rank; ++j)
+        if (f->in.rep_shape[j] != f->out.rep_shape[j])
+            return fail(AOL_E_SHAPE, "input and output repetition spaces differ");
+    const int64_t n_in = elems(f->in.pattern_shape, f->in.pattern_rank);
+    const int64_t n_out = elems(f->out.pattern_shape, f->out.pattern_rank);
+    if (n_in > AOL_MAX_FILTER_PATTERN) return fail(AOL_E_RANGE, "input pattern larger than AOL_MAX_FILTER_PATTERN");
+    if (f->n_windows < 1 || f->n_windows > AOL_MAX_WINDOWS || n_out != f->n_windows)
+        return fail(AOL_E_SHAPE, "n_windows must equal the output pattern size (1..AOL_MAX_WINDOWS)");
+    if (f->window_len < 1 || f->divisor == 0) return fail(AOL_E_INVALID, "window_len >= 1 and divisor != 0");
+    for (int k = 0; k < f->n_windows; ++k)
+        if (f->window_start[k] < 0 || int64_t(f->window_start[k]) + f->window_len > n_in)
+            return fail(AOL_E_SHAPE, "window outside the input pattern");
+    for (const aol_tiler_t* t : {&f->in, &f->out}) {
+        for (int a = 0; a < t->array_rank; ++a)
+            if (t->array_shape[a] >= (int64_t(1) << 31)) return fail(AOL_E_RANGE, "filter array extents must be < 2^31");
+        if (elems(t->array_shape, t->array_rank) >= (int64_t(1) << 62)) return fail(AOL_E_RANGE, "array too large");
+    }
+    return AOL_OK;
+}
+
+void fill_side(const aol_tiler_t* t, int32_t* s, int64_t* st, int32_t* o, int32_t (*P)[AOL_MAX_RANK]) {
+    int64_t stride = 1;
+    for (int a = t->array_rank - 1; a >= 0; --a) {
+        s[a] = int32_t(t->array_shape[a]);
+        st[a] = stride;
+        stride *= t->array_shape[a];
+        o[a] = int32_t(emod(t->origin[a], t->array_shape[a]));
+        for (int j = 0; j < t->rep_rank; ++j) P[a][j] = int32_t(emod(t->paving[a][j], t->array_shape[a]));
+    }
+}
+
+void fill_offsets(const aol_tiler_t* t, int64_t n, int32_t (*f)[AOL_MAX_RANK]) {
+    for (int64_t p = 0; p < n; ++p) {
+        int64_t idx[AOL_MAX_RANK] = {0};
+        unflatten(p, t->pattern_shape, t->pattern_rank, idx);
+        for (int a = 0; a < t->array_rank; ++a) {
+            __int128 v = 0;
+            for (int k = 0; k < t->pattern_rank; ++k) v += __int128(emod(t->fitting[a][k], t->array_shape[a])) * idx[k];
+            f[p][a] = int32_t(v % t->array_shape[a]);
+        }
+    }
+}
+
+}  // namespace
+
+}  // namespace aol
+
+using namespace aol;
+
+extern "C" {
+
+aol_status_t aol_filter_validate(const aol_filter_t* f) { return check_filter(f); }
+
+aol_status_t aol_filter_preset(aol_filter_kind_t which, int64_t planes, int64_t H, int64_t W, aol_filter_t* out) {
+    if (!out) return fail(AOL_E_INVALID, "out is NULL");
+    if (planes <= 0 || H <= 0 || W <= 0) return fail(AOL_E_INVALID, "planes, H, W must be > 0");
+    aol_filter_t f;
+    std::memset(&f, 0, sizeof f);
+    // the per-plane tilers of Fig. 10 (H) / reading Z1 (V), lifted to a stack of planes:
+    // array {planes, ...}, repetition {planes, ...}, paving 1 on the plane dimension
+    aol_tiler_t tin, tout;
+    aol_status_t st;
+    if (which == AOL_FILTER_H) {
+        if ((st = aol_tiler_preset(AOL_PRESET_H_IN, H, W, &tin)) != AOL_OK) return st;
+        if ((st = aol_tiler_preset(AOL_PRESET_H_OUT, H, W, &tout)) != AOL_OK) return st;
+        f.n_windows = 3;
+        const int32_t s[3] = {0, 2, 5};   // Fig. 5: tmp0 over [0..5], tmp1 over [2..7], tmp2 over [5..10]
+        for (int k = 0; k < 3; ++k) f.window_start[k] = s[k];
+    } else if (which == AOL_FILTER_V) {
+        if ((st = aol_tiler_preset(AOL_PRESET_V_IN, H, W, &tin)) != AOL_OK) return st;
+        if ((st = aol_tiler_preset(AOL_PRESET_V_OUT, H, W, &tout)) != AOL_OK) return st;
+        f.n_windows = 4;
+        const int32_t s[4] = {0, 2, 4, 6};   // reading Z1
+        for (int k = 0; k < 4; ++k) f.window_start[k] = s[k];
+    } else {
+        return fail(AOL_E_INVALID, "unknown filter kind");
+    }
+    f.window_len = 6;
+    f.divisor = 6;
+    for (aol_tiler_t* t : {&tin, &tout}) {
+        aol_tiler_t l;
+        std::memset(&l, 0, sizeof l);
+        l.array_rank = 3;
+        l.rep_rank = 3;
+        l.pattern_rank = t->pattern_rank;
+        l.array_shape[0] = planes;
+        l.rep_shape[0] = planes;
+        l.paving[0][0] = 1;
+        for (int a = 0; a < 2; ++a) {
+            l.array_shape[a + 1] = t->array_shape[a];
+            l.origin[a + 1] = t->origin[a];
+            for (int j = 0; j < 2; ++j) l.paving[a + 1][j + 1] = t->paving[a][j];
+            for (int k = 0; k < t->pattern_rank; ++k) l.fitting[a + 1][k] = t->fitting[a][k];
+        }
+        for (int j = 0; j < 2; ++j) l.rep_shape[j + 1] = t->rep_shape[j];
+        for (int k = 0; k < t->pattern_rank; ++k) l.pattern_shape[k] = t->pattern_shape[k];
+        *t = l;
+    }
+    f.in = tin;
+    f.out = tout;
+    *out = f;
+    return AOL_OK;
+}
+
+aol_status_t aol_filter_apply(const aol_filter_t* f, const int32_t* d_in, int32_t* d_out, cudaStream_t s) {
+    aol_status_t st = check_filter(f);
+    if (st != AOL_OK) return st;
+    if (!d_in || !d_out) return fail(AOL_E_INVALID, "null buffer");
+    if ((reinterpret_cast<uintptr_t>(d_in) | reinterpret_cast<uintptr_t>(d_out)) % 4)
+        return fail(AOL_E_ALIGN, "buffers must be 4-byte aligned");
+    FilterDev fd;
+    std::memset(&fd, 0, sizeof fd);
+    fd.ra_in = f->in.array_rank;
+    fd.ra_out = f->out.array_rank;
+    fd.rr = f->in.rep_rank;
+    fd.n_in = int32_t(elems(f->in.pattern_shape, f->in.pattern_rank));
+    fd.n_win = f->n_windows;
+    fd.len = f->window_len;
+    fd.divisor = f->divisor;
+    fd.nrep = elems(f->in.rep_shape, f->in.rep_rank);
+    if (fd.nrep == 0) return AOL_OK;
+    fd.fast32 = fd.nrep < (int64_t(1) << 31);
+    for (int j = 0; j < fd.rr; ++j) {
+        fd.rep_ext[j] = int32_t(std::min<int64_t>(f->in.rep_shape[j], INT32_MAX));
+        if (f->in.rep_shape[j] >= (int64_t(1) << 31)) fd.fast32 = 0;
+    }
+    for (int j = 0; j < fd.rr; ++j) {
+        uint32_t shift = 0;
+        while (shift < 32 && (uint64_t(1) << shift) < uint64_t(fd.rep_ext[j])) ++shift;
+        fd.fd_shift[j] = shift;
+        fd.fd_mul[j] = uint32_t(((uint64_t(1) << 32) * ((uint64_t(1) << shift) - uint64_t(fd.rep_ext[j]))) /
+                                    uint64_t(fd.rep_ext[j]) + 1);
+    }
+    fill_side(&f->in, fd.s_in, fd.st_in, fd.o_in, fd.P_in);
+    fill_side(&f->out, fd.s_out, fd.st_out, fd.o_out, fd.P_out);
+    for (int k = 0; k < fd.n_win; ++k) fd.start[k] = f->window_start[k];
+    fill_offsets(&f->in, fd.n_in, fd.f_in);
+    fill_offsets(&f->out, fd.n_win, fd.f_out);
+
+    DeviceInfo dev;
+    st = device_info(&dev);
+    if (st != AOL_OK) return st;
+    const int grid = int(std::max<int64_t>(1, std::min<int64_t>((fd.nrep + 255) / 256, int64_t(dev.num_sms) * 16)));
+    if (fd.fast32)
+        filter_kernel<true><<<grid, 256, 0, s>>>(fd, d_in, d_out);
+    else
+        filter_kernel<false><<<grid, 256, 0, s>>>(fd, d_in, d_out);
+    AOL_LAUNCH_CHECK("filter_kernel");
+    return AOL_OK;
+}
+
+}  // extern "C"

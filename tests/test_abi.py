@@ -167,6 +167,35 @@ def test_package_has_no_oracle_dependency():
                 assert "import oracle" not in src and "from oracle" not in src and "aol_oracle" not in src, fn
 
 
+def test_filter_presets_and_validation(orc):
+    """f3 filters: the presets lift the oracle's per-plane tilers to a stack of planes."""
+    for kind, which_in, which_out, Wv in ((aol.FILTER_H, 0, 1, 64), (aol.FILTER_V, 2, 3, 24)):
+        f = aol.filter_preset(kind, 5, 18, Wv)
+        aol.filter_validate(f)
+        for side, which in ((f.in_, which_in), (f.out, which_out)):
+            arr, rep, pat = aol._shapes(side)
+            o = orc.preset(which, 18, Wv)
+            oarr, orep, opat = o.shapes
+            assert arr == (5,) + oarr and rep == (5,) + orep and pat == opat
+            assert side.paving[0][0] == 1 and all(side.paving[a + 1][j + 1] == o.paving[a][j]
+                                                  for a in range(2) for j in range(2))
+    f = aol.filter_preset(aol.FILTER_H, 1, 9, 16)
+    bad = [("divisor", 0, _lib.E_INVALID), ("window_len", 0, _lib.E_INVALID), ("n_windows", 4, _lib.E_SHAPE)]
+    for field, val, code in bad:
+        g = aol.filter_preset(aol.FILTER_H, 1, 9, 16)
+        setattr(g, field, val)
+        with pytest.raises(aol.AolError) as e:
+            aol.filter_validate(g)
+        assert e.value.status == code, field
+    g = aol.filter_preset(aol.FILTER_H, 1, 9, 16)
+    g.out.rep_shape[1] = 3
+    with pytest.raises(aol.AolError):
+        aol.filter_validate(g)
+    with pytest.raises(aol.AolError):
+        aol.filter_preset(aol.FILTER_V, 1, 10, 16)
+    assert f.n_windows == 3 and list(f.window_start)[:3] == [0, 2, 5] and f.window_len == 6
+
+
 def test_kernel_division_identities():
     """The kernels rewrite Fig. 5's tmp/6 - tmp%6 (C semantics) as 7*(tmp/6) - tmp, and for
     non-negative 8-bit sums use tmp/6 == (tmp*43691) >> 18 (32-bit).  Both are checked

@@ -244,6 +244,54 @@ def test_tiler_linear_paths(orc, case, dtype):
         assert np.array_equal(arr_t.cpu().numpy(), So), mode
 
 
+@pytest.mark.parametrize("shape", [(3, 1080, 1920), (4, 288, 352), (2, 9, 8), (3, 27, 1000)])
+def test_filter_presets_vs_oracle(orc, shape):
+    """f3: the run-time generic repetition (gather + task + scatter in one kernel) with the paper's
+    H and V descriptions equals the oracle's three-step filters."""
+    P, H, W = shape
+    xh = synth.frames(41, 0, 1, P, H, W, "signed")[0] >> 6
+    x = torch.from_numpy(xh).cuda()
+    y = aol.filter_apply(aol.filter_preset(aol.FILTER_H, P, H, W), x)
+    torch.cuda.synchronize()
+    yo = orc.downscale_h(xh)
+    assert np.array_equal(y.cpu().numpy(), yo)
+    z = aol.filter_apply(aol.filter_preset(aol.FILTER_V, P, H, 3 * W // 8), y)
+    torch.cuda.synchronize()
+    assert np.array_equal(z.cpu().numpy(), orc.downscale_v(yo))
+
+
+@pytest.mark.parametrize("seed", range(30))
+def test_filter_random_tilers_vs_oracle(orc, seed):
+    """f3 with random input/output tilers and the paper's task windows: equal to the oracle's
+    gather -> task_h/task_v -> scatter (Fig. 4, 5, 6) on the same descriptors."""
+    rng = np.random.default_rng(900 + seed)
+    n_in, starts, task = ((11, [0, 2, 5], orc.task_h) if seed % 2 == 0 else (12, [0, 2, 4, 6], orc.task_v))
+    n_out = len(starts)
+    ra = int(rng.integers(1, 4))
+    rep = [int(rng.integers(1, 6)) for _ in range(int(rng.integers(1, 3)))]
+    arr_in = [int(rng.integers(2, 17)) for _ in range(ra)]
+    o_in = [int(rng.integers(-2 * s, 2 * s + 1)) for s in arr_in]
+    P_in = [[int(rng.integers(-4, 10)) for _ in rep] for _ in range(ra)]
+    F_in = [[int(rng.integers(-4, 10))] for _ in range(ra)]
+    # injective output tiler: array [prod(rep), n_out], row = flattened rep, col = k
+    nrep = int(np.prod(rep))
+    arr_out = [nrep, n_out]
+    strides = [int(np.prod(rep[j + 1:])) for j in range(len(rep))]
+    P_out = [strides, [0] * len(rep)]
+    F_out = [[0], [1]]
+    xh = np.asarray(rng.integers(-300, 300, size=arr_in)).astype(np.int32)
+    oti = orc.make_tiler(arr_in, rep, [n_in], o_in, P_in, F_in)
+    oto = orc.make_tiler(arr_out, rep, [n_out], [0, 0], P_out, F_out)
+    bg = np.full(arr_out, -99, np.int32)
+    want = orc.scatter(oto, task(orc.gather(oti, xh)), bg)
+    f = aol.make_filter(aol.make_tiler(arr_in, rep, [n_in], o_in, P_in, F_in),
+                        aol.make_tiler(arr_out, rep, [n_out], [0, 0], P_out, F_out), starts, 6, 6)
+    out = torch.from_numpy(bg.copy()).cuda()
+    aol.filter_apply(f, torch.from_numpy(xh).cuda(), out=out)
+    torch.cuda.synchronize()
+    assert np.array_equal(out.cpu().numpy(), want)
+
+
 def test_tiler_paper_presets_on_gpu(orc):
     H, W = 27, 64
     xh = synth.planes(4, 1, H, W)[0]

@@ -139,6 +139,24 @@ def main():
               "check_gather_is_blocking": bool(torch.equal(G[1, 2, 3], A[1, 16:24, 24:32]))})
         del A, G, B
         torch.cuda.empty_cache()
+    if want("f3"):
+        # the paper's generic-vs-non-generic experiment on B200: run-time descriptors,
+        # one fused gather+task+scatter kernel per filter, Y through HBM between the two filters
+        N, C, H, W = 300, 3, 1080, 1920
+        x = aol.synth_frames(0, 0, N, C, H, W).reshape(N * C, H, W)
+        fh = aol.filter_preset(aol.FILTER_H, N * C, H, W)
+        fv = aol.filter_preset(aol.FILTER_V, N * C, H, 720)
+        y = torch.empty((N * C, H, 720), dtype=torch.int32, device="cuda")
+        z = torch.empty((N * C, 480, 720), dtype=torch.int32, device="cuda")
+        th, _ = timed(lambda: aol.filter_apply(fh, x, out=y), reps=5)
+        tv, _ = timed(lambda: aol.filter_apply(fv, y, out=z), reps=5)
+        zf, _ = aol.downscale_frame(x.reshape(N, C, H, W))
+        b = frames_bytes(N, C, H, W)
+        emit({"config": "f3 generic run-time filters H then V (300 HD frames)", "h_ms": th, "v_ms": tv,
+              "frames_per_s": N / ((th + tv) / 1e3), "GBps_algorithmic": b / ((th + tv) / 1e3) / 1e9,
+              "equals_fused": bool(torch.equal(zf.reshape(N * C, 480, 720), z))})
+        del x, y, z, zf
+        torch.cuda.empty_cache()
     if want("d4"):
         fused_line("d4 4K batch", 64, 3, 2160, 3840)
     if want("f1"):

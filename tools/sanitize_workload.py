@@ -1,0 +1,61 @@
+#!/usr/bin/env python
+"""Small launches of every kernel, for compute-sanitizer (memcheck / racecheck / synccheck / initcheck).
+
+Exits non-zero if any result differs from a second computation path, so a sanitizer run also checks
+that instrumented execution still produces the right answer.
+"""
+import os
+import sys
+
+import torch
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+sys.path.insert(0, ROOT)
+import paper_conf_ipps_guortgbs11_b200 as aol  # noqa: E402
+
+
+def main():
+    torch.cuda.set_device(0)
+    ok = True
+    for (N, C, H, W) in [(2, 3, 27, 64), (1, 1, 9, 32), (1, 2, 18, 352)]:
+        for dt in (torch.int32, torch.uint8):
+            x = aol.synth_frames(1, 0, N, C, H, W, "uniform", dtype=dt)
+            ref = None
+            for opts in ({"kernel": 2}, {"kernel": 1}, {"kernel": 1, "stages": 2, "bands_per_unit": 1},
+                         {"kernel": 1, "ctas_per_sm": 2}, {"kernel": 1, "flags": 1}):
+                try:
+                    z, cs = aol.downscale_frame(x, checksums=True, opts=opts)
+                except aol.AolError:
+                    continue   # shape not eligible for this kernel
+                torch.cuda.synchronize()
+                if ref is None:
+                    ref = (z.clone(), cs.clone())
+                else:
+                    ok &= torch.equal(z, ref[0]) and torch.equal(cs.view(torch.int64), ref[1].view(torch.int64))
+        x = aol.synth_frames(2, 0, N, C, H, W, "signed")
+        y = aol.downscale_h(x)
+        z = aol.downscale_v(y)
+        zf, _ = aol.downscale_frame(x)
+        ok &= torch.equal(z, zf)
+        ok &= torch.equal(aol.frame_checksum(z).view(torch.int64),
+                          aol.downscale_frame(x, checksums=True)[1].view(torch.int64))
+    t = aol.make_tiler([16, 24], [2, 3], [8, 8], [0, 0], [[8, 0], [0, 8]], [[1, 0], [0, 1]])
+    A = torch.arange(16 * 24, dtype=torch.int32, device="cuda").reshape(16, 24)
+    G = aol.tiler_gather(t, A)
+    B = torch.zeros_like(A)
+    aol.tiler_scatter(t, G, B, mode="fast")
+    ok &= torch.equal(A, B)
+    B.zero_()
+    aol.tiler_scatter(t, G, B, mode="sequential")
+    ok &= torch.equal(A, B)
+    tw = aol.make_tiler([9, 10], [4], [5, 3], [-3, 7], [[2], [3]], [[1, 0], [0, -1]])   # wrapping
+    G2 = aol.tiler_gather(tw, A[:9, :10].contiguous())
+    C2 = torch.zeros((9, 10), dtype=torch.int32, device="cuda")
+    aol.tiler_scatter(tw, G2, C2, mode="sequential")
+    torch.cuda.synchronize()
+    print("sanitize workload:", "OK" if ok else "MISMATCH")
+    return 0 if ok else 1
+
+
+if __name__ == "__main__":
+    sys.exit(main())
