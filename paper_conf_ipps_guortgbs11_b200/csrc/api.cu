@@ -147,6 +147,38 @@ aol_status_t make_tiler_dev(const aol_tiler_t* t, TilerDev* td) {
         td->fd_mul[d] = td->fast32 ? uint32_t(magic) : 0u;
         td->fd_shift[d] = shift;
     }
+    // Walk order for linear tilers: array-side strides ascending (innermost = smallest), dims that
+    // do not move on the array side (stride 0, broadcast) outermost; the natural last dim stays
+    // innermost when it is unit-stride on the array side so 16-byte vectors remain possible.
+    int order[2 * AOL_MAX_RANK];
+    for (int d = 0; d < td->nd; ++d) order[d] = d;
+    if (td->linear) {
+        auto key = [&](int d) { return td->lin[d] == 0 ? INT64_MAX : td->lin[d]; };
+        // stable insertion sort, descending key = outermost first
+        for (int i = 1; i < td->nd; ++i)
+            for (int j = i; j > 0 && key(order[j - 1]) < key(order[j]); --j) std::swap(order[j - 1], order[j]);
+        const int last = td->nd - 1;
+        if (td->nd > 0 && td->lin[last] == 1) {
+            int pos = 0;
+            while (order[pos] != last) ++pos;
+            for (; pos < last; ++pos) order[pos] = order[pos + 1];
+            order[last] = last;
+        }
+    }
+    int64_t gst[2 * AOL_MAX_RANK];
+    int64_t g = 1;
+    for (int d = td->nd - 1; d >= 0; --d) {
+        gst[d] = g;
+        g *= td->ext[d];
+    }
+    for (int i = 0; i < td->nd; ++i) {
+        const int d = order[i];
+        td->p_ext[i] = td->ext[d];
+        td->p_lin[i] = td->lin[d];
+        td->p_gst[i] = gst[d];
+        td->p_fd_mul[i] = td->fd_mul[d];
+        td->p_fd_shift[i] = td->fd_shift[d];
+    }
     return AOL_OK;
 }
 

@@ -83,6 +83,11 @@ struct TilerDev {
     int64_t lin[2 * AOL_MAX_RANK];  // element offset per unit of combined index d (linear tilers)
     int64_t base;                   // element offset of the origin
     uint32_t fd_mul[2 * AOL_MAX_RANK], fd_shift[2 * AOL_MAX_RANK];
+    // Linear tilers are walked in an order that makes the ARRAY side contiguous (dims sorted by
+    // array stride, smallest innermost); p_* describe the permuted dims: extent, array stride,
+    // tile stride (row-major over the natural [rep..., pattern...] order) and magic divisors.
+    int64_t p_ext[2 * AOL_MAX_RANK], p_lin[2 * AOL_MAX_RANK], p_gst[2 * AOL_MAX_RANK];
+    uint32_t p_fd_mul[2 * AOL_MAX_RANK], p_fd_shift[2 * AOL_MAX_RANK];
     int64_t total;              // rep elements * pattern elements
     int64_t array_elems;
 };

@@ -11,9 +11,12 @@
 // index -- offset = base + sum_d lin[d] * idx[d] -- and the LINEAR kernels
 // apply: one fast 32-bit division chain per thread and, when the innermost
 // pattern dimension walks contiguous memory, 16-byte vector accesses on both
-// sides.  Otherwise the GENERAL kernels evaluate the modulo per wrapping
-// dimension.  Tile-side accesses are always coalesced (consecutive threads,
-// consecutive tile elements).
+// sides.  Linear tilers are walked in array-stride order (the host sorts the
+// combined dims so consecutive threads touch consecutive ARRAY addresses, the
+// side whose locality is not guaranteed); the tile side is then written in
+// contiguous runs of the innermost dim.  Otherwise the GENERAL kernels walk the
+// natural tile order (tile accesses coalesced) and evaluate the modulo per
+// wrapping dimension.
 #include <cuda_runtime.h>
 
 #include <algorithm>
@@ -69,34 +72,27 @@ struct Vec<16> {
 
 constexpr int kND = 2 * AOL_MAX_RANK;
 
-// Decompose flat tile index g into the combined (rep ++ pattern) multi-index, last dim fastest.
+// Decompose flat index g over extents ext (last dim fastest).
 template <bool kFast32>
-__device__ __forceinline__ void decompose(const TilerDev& td, int64_t g, int64_t (&idx)[kND]) {
+__device__ __forceinline__ void decompose(int nd, const int64_t* ext, const uint32_t* fmul, const uint32_t* fshift,
+                                          int64_t g, int64_t (&idx)[kND]) {
 #pragma unroll
     for (int d = kND - 1; d >= 0; --d) {
-        if (d < td.nd) {
+        if (d < nd) {
             if (kFast32) {
                 const uint32_t n = uint32_t(g);
-                const uint32_t q = (__umulhi(n, td.fd_mul[d]) + n) >> td.fd_shift[d];
-                idx[d] = int64_t(n - q * uint32_t(td.ext[d]));
+                const uint32_t q = (__umulhi(n, fmul[d]) + n) >> fshift[d];
+                idx[d] = int64_t(n - q * uint32_t(ext[d]));
                 g = q;
             } else {
-                const int64_t q = g / td.ext[d];
-                idx[d] = g - q * td.ext[d];
+                const int64_t q = g / ext[d];
+                idx[d] = g - q * ext[d];
                 g = q;
             }
         } else {
             idx[d] = 0;
         }
     }
-}
-
-__device__ __forceinline__ int64_t linear_offset(const TilerDev& td, const int64_t (&idx)[kND]) {
-    int64_t off = td.base;
-#pragma unroll
-    for (int d = 0; d < kND; ++d)
-        if (d < td.nd) off += td.lin[d] * idx[d];
-    return off;
 }
 
 __device__ __forceinline__ int64_t general_offset(const TilerDev& td, const int64_t (&idx)[kND]) {
@@ -123,20 +119,73 @@ __global__ void __launch_bounds__(256) tiler_kernel(const TilerDev td, const voi
     using T = typename Elem<ES>::T;
     using VT = typename Vec<ES * V>::T;
     const int64_t nvec = td.total / V;
-    for (int64_t v = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; v < nvec; v += int64_t(gridDim.x) * blockDim.x) {
-        const int64_t g = v * V;
-        int64_t idx[kND];
-        decompose<kFast32>(td, g, idx);
-        const int64_t off = kLinear ? linear_offset(td, idx) : general_offset(td, idx);
+    const int64_t stride = int64_t(gridDim.x) * blockDim.x;
+    // kU independent elements per thread per iteration: all loads issued before the stores, so each
+    // thread keeps kU requests in flight (Little's law at ~43 GB/s per SM needs tens of KB per SM).
+    constexpr int kU = (MODE <= 1) ? 4 : 1;
+    // a warp owns kU*32 consecutive vectors per iteration (lane + 32u): locality is kept on both sides
+    const int64_t warp_first = (int64_t(blockIdx.x) * blockDim.x + (threadIdx.x & ~31u)) * kU + (threadIdx.x & 31u);
+    for (int64_t v0 = warp_first; v0 < nvec; v0 += kU * stride) {
+        int64_t off[kU], g[kU];   // array-side and tile-side element offsets
+#pragma unroll
+        for (int u = 0; u < kU; ++u) {
+            const int64_t v = v0 + 32 * u;
+            if (kLinear) {
+                // permuted walk (array side contiguous): both offsets are affine in the permuted index;
+                // a runtime-rank loop that folds each digit straight into the two offsets (no index array)
+                int64_t o = td.base, gg = 0;
+                if (kFast32) {
+                    uint32_t n = v < nvec ? uint32_t(v * V) : 0u;
+#pragma unroll 1
+                    for (int d = td.nd - 1; d >= 0; --d) {
+                        const uint32_t q = (__umulhi(n, td.p_fd_mul[d]) + n) >> td.p_fd_shift[d];
+                        const uint32_t i = n - q * uint32_t(td.p_ext[d]);
+                        n = q;
+                        o += td.p_lin[d] * int64_t(i);
+                        gg += td.p_gst[d] * int64_t(i);
+                    }
+                } else {
+                    int64_t n = v < nvec ? v * V : 0;
+#pragma unroll 1
+                    for (int d = td.nd - 1; d >= 0; --d) {
+                        const int64_t q = n / td.p_ext[d];
+                        const int64_t i = n - q * td.p_ext[d];
+                        n = q;
+                        o += td.p_lin[d] * i;
+                        gg += td.p_gst[d] * i;
+                    }
+                }
+                off[u] = o;
+                g[u] = gg;
+            } else {
+                int64_t idx[kND];
+                g[u] = v < nvec ? v * V : 0;
+                decompose<kFast32>(td.nd, td.ext, td.fd_mul, td.fd_shift, g[u], idx);
+                off[u] = general_offset(td, idx);
+            }
+        }
         if (MODE == 0) {
             // tiles[g .. g+V) = array[off .. off+V)   (V > 1 only when contiguous and aligned)
-            reinterpret_cast<VT*>(dst)[v] = reinterpret_cast<const VT*>(static_cast<const T*>(src) + off)[0];
+            VT val[kU];
+#pragma unroll
+            for (int u = 0; u < kU; ++u)
+                if (v0 + 32 * u < nvec) val[u] = reinterpret_cast<const VT*>(static_cast<const T*>(src) + off[u])[0];
+#pragma unroll
+            for (int u = 0; u < kU; ++u)
+                if (v0 + 32 * u < nvec) reinterpret_cast<VT*>(static_cast<T*>(dst) + g[u])[0] = val[u];
         } else if (MODE == 1) {
-            reinterpret_cast<VT*>(static_cast<T*>(dst) + off)[0] = reinterpret_cast<const VT*>(src)[v];
+            VT val[kU];
+#pragma unroll
+            for (int u = 0; u < kU; ++u)
+                if (v0 + 32 * u < nvec) val[u] = reinterpret_cast<const VT*>(static_cast<const T*>(src) + g[u])[0];
+#pragma unroll
+            for (int u = 0; u < kU; ++u)
+                if (v0 + 32 * u < nvec) reinterpret_cast<VT*>(static_cast<T*>(dst) + off[u])[0] = val[u];
         } else if (MODE == 2) {
-            atomicMax(ws + off, (unsigned long long)g + 1ull);
+            atomicMax(ws + off[0], (unsigned long long)g[0] + 1ull);
         } else {
-            if (ws[off] == (unsigned long long)g + 1ull) static_cast<T*>(dst)[off] = static_cast<const T*>(src)[g];
+            if (ws[off[0]] == (unsigned long long)g[0] + 1ull)
+                static_cast<T*>(dst)[off[0]] = static_cast<const T*>(src)[g[0]];
         }
     }
 }
@@ -187,14 +236,15 @@ aol_status_t launch_mode(const TilerDev& td, int elsize, int vec, const void* sr
     return fail(AOL_E_DTYPE, "element size must be 1, 2, 4 or 8 bytes");
 }
 
-// Largest usable vector (elements): contiguous innermost dim, divisibility and alignment.
+// Largest usable vector (elements): the permuted innermost dim is the natural last dim, unit-stride on
+// both sides; every other stride, the origin and the pointers keep V-element alignment.
 int vector_width(const TilerDev& td, int elsize, const void* p_array, const void* p_tiles) {
     const int v = 16 / elsize;
     if (!td.linear || td.nd == 0 || v <= 1) return 1;
     const int last = td.nd - 1;
-    if (td.lin[last] != 1 || td.ext[last] % v != 0 || td.base % v != 0) return 1;
+    if (td.p_lin[last] != 1 || td.p_gst[last] != 1 || td.p_ext[last] % v != 0 || td.base % v != 0) return 1;
     for (int d = 0; d < last; ++d)
-        if (td.lin[d] % v != 0) return 1;
+        if (td.p_lin[d] % v != 0 || td.p_gst[d] % v != 0) return 1;
     if ((reinterpret_cast<uintptr_t>(p_array) | reinterpret_cast<uintptr_t>(p_tiles)) % 16) return 1;
     return v;
 }
