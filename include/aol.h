@@ -15,8 +15,10 @@
  *
  * Conventions for every entry point:
  *  - Device pointers ("d_") are owned by the caller (e.g. PyTorch); the library
- *    allocates no device memory and holds no global state other than a
- *    thread-local error string, so it is re-entrant.
+ *    allocates no device memory.  Its only global state is a thread-local
+ *    error string and mutex-guarded memos of immutable per-process facts
+ *    (device attributes, kernel attributes it set, occupancy), so it is
+ *    re-entrant and thread-safe.
  *  - Device calls are stream-ordered on the given stream and return after
  *    launch (asynchronous).  Kernel faults surface at the caller's next sync.
  *  - Errors are returned synchronously as aol_status_t for invalid arguments,

@@ -6,7 +6,9 @@
 #include <cstdarg>
 #include <cstdint>
 #include <cstring>
+#include <mutex>
 #include <string>
+#include <unordered_map>
 #include <vector>
 
 #include "common.h"
@@ -30,14 +32,74 @@ void clear_error() { g_err.clear(); }
 
 const char* last_error_cstr() { return g_err.c_str(); }
 
+// Immutable per-process facts (device attributes, kernel attributes the library has set, occupancy
+// of a kernel configuration) are memoised: they never change for a process, and querying them on
+// every call made the host side of a launch several microseconds longer than a one-frame kernel.
+namespace {
+std::mutex g_cache_mu;
+std::unordered_map<int, DeviceInfo> g_dev_cache;
+std::unordered_map<std::string, int> g_kernel_cache;   // "dev:fn:smem" -> applied, "dev:fn:block:smem" -> occ
+
+std::string key_of(int dev, const void* fn, int a, int b) {
+    char buf[96];
+    snprintf(buf, sizeof buf, "%d:%p:%d:%d", dev, fn, a, b);
+    return buf;
+}
+}  // namespace
+
 aol_status_t device_info(DeviceInfo* out) {
     int dev = 0;
     AOL_CUDA_TRY(cudaGetDevice(&dev));
-    out->device = dev;
-    AOL_CUDA_TRY(cudaDeviceGetAttribute(&out->num_sms, cudaDevAttrMultiProcessorCount, dev));
-    AOL_CUDA_TRY(cudaDeviceGetAttribute(&out->smem_optin, cudaDevAttrMaxSharedMemoryPerBlockOptin, dev));
-    AOL_CUDA_TRY(cudaDeviceGetAttribute(&out->smem_per_sm, cudaDevAttrMaxSharedMemoryPerMultiprocessor, dev));
+    {
+        std::lock_guard<std::mutex> lk(g_cache_mu);
+        auto it = g_dev_cache.find(dev);
+        if (it != g_dev_cache.end()) {
+            *out = it->second;
+            return AOL_OK;
+        }
+    }
+    DeviceInfo d;
+    d.device = dev;
+    AOL_CUDA_TRY(cudaDeviceGetAttribute(&d.num_sms, cudaDevAttrMultiProcessorCount, dev));
+    AOL_CUDA_TRY(cudaDeviceGetAttribute(&d.smem_optin, cudaDevAttrMaxSharedMemoryPerBlockOptin, dev));
+    AOL_CUDA_TRY(cudaDeviceGetAttribute(&d.smem_per_sm, cudaDevAttrMaxSharedMemoryPerMultiprocessor, dev));
+    std::lock_guard<std::mutex> lk(g_cache_mu);
+    g_dev_cache[dev] = d;
+    *out = d;
     return AOL_OK;
+}
+
+aol_status_t kernel_smem(const void* fn, int smem) {
+    // the attribute is an upper bound: only ever raise it, and remember the largest value applied
+    int dev = 0;
+    AOL_CUDA_TRY(cudaGetDevice(&dev));
+    const std::string k = key_of(dev, fn, -1, -1);
+    std::lock_guard<std::mutex> lk(g_cache_mu);
+    auto it = g_kernel_cache.find(k);
+    if (it != g_kernel_cache.end() && it->second >= smem) return AOL_OK;
+    AOL_CUDA_TRY(cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, smem));
+    g_kernel_cache[k] = smem;
+    return AOL_OK;
+}
+
+int kernel_occupancy(const void* fn, int block, int smem) {
+    int dev = 0;
+    if (cudaGetDevice(&dev) != cudaSuccess) return 0;
+    const std::string k = key_of(dev, fn, block, smem);
+    {
+        std::lock_guard<std::mutex> lk(g_cache_mu);
+        auto it = g_kernel_cache.find(k);
+        if (it != g_kernel_cache.end()) return it->second;
+    }
+    int occ = 0;
+    if (kernel_smem(fn, smem) != AOL_OK ||
+        cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, fn, block, smem) != cudaSuccess) {
+        (void)cudaGetLastError();
+        return 0;
+    }
+    std::lock_guard<std::mutex> lk(g_cache_mu);
+    g_kernel_cache[k] = occ;
+    return occ;
 }
 
 int elsize_of(aol_dtype_t el) {

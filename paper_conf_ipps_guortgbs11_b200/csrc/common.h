@@ -10,7 +10,7 @@
 
 namespace aol {
 
-// Thread-local last-error message (the library's only mutable state).
+// Thread-local last-error message (besides the memos in api.cu, the library's only mutable state).
 void set_error(const char* fmt, ...) __attribute__((format(printf, 1, 2)));
 void clear_error();
 
@@ -48,7 +48,9 @@ struct DeviceInfo {
     int smem_optin;   // max dynamic smem per block (opt-in)
     int smem_per_sm;  // shared memory per multiprocessor
 };
-aol_status_t device_info(DeviceInfo* out);
+aol_status_t device_info(DeviceInfo* out);               // memoised per device
+aol_status_t kernel_smem(const void* fn, int smem_bytes);   // cudaFuncSetAttribute(MaxDynamicSmem), memoised
+int kernel_occupancy(const void* fn, int block, int smem);  // resident CTAs per SM, memoised (0 on error)
 
 // ---- launchers implemented in the .cu files (all validate nothing; callers do)
 struct FusedPlan {

@@ -94,16 +94,8 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, const void* d_in, const int32_t* d
             }
             int occ = 0;
             const int smem = stages * int(stage_stride) + kOutBufs * int(out_bytes) + 2 * stages * 8 + 1024;
-            if (stages >= 2) {
-                KernelFn k = pick(in_dtype, true, block, cps);
-                if (cudaFuncSetAttribute(reinterpret_cast<const void*>(k), cudaFuncAttributeMaxDynamicSharedMemorySize,
-                                         smem) != cudaSuccess ||
-                    cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, reinterpret_cast<const void*>(k), block,
-                                                                  smem) != cudaSuccess) {
-                    (void)cudaGetLastError();
-                    occ = 0;
-                }
-            }
+            if (stages >= 2 && cps > 1) occ = kernel_occupancy(reinterpret_cast<const void*>(pick(in_dtype, true, block, cps)), block, smem);
+            if (cps == 1) occ = 1;   // one CTA always fits once its shared memory does
             if ((stages >= 2 && occ >= cps) || cps == 1 || o.ctas_per_sm > 0) {
                 if (stages < 2) tma_ok = false;
                 break;
@@ -221,8 +213,8 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
     a.halo_last = (plan.flags & AOL_FLAG_HALO_LAST) ? 1 : 0;
 
     KernelFn k = pick(in_dtype, d_cs != nullptr, plan.block, plan.ctas_per_sm);
-    AOL_CUDA_TRY(cudaFuncSetAttribute(reinterpret_cast<const void*>(k), cudaFuncAttributeMaxDynamicSharedMemorySize,
-                                      plan.smem));
+    aol_status_t st_attr = kernel_smem(reinterpret_cast<const void*>(k), plan.smem);
+    if (st_attr != AOL_OK) return st_attr;
     k<<<plan.grid, plan.block, plan.smem, s>>>(map, a);
     AOL_LAUNCH_CHECK("fused_tma_kernel");
     return AOL_OK;
