@@ -104,11 +104,12 @@ typedef struct {
     int32_t bands_per_unit; /* 9-row bands per work unit, 0 = auto (balance waves vs halo)     */
     int32_t kernel;         /* 0 = auto, 1 = TMA fused kernel (error if shape unsupported),
                                2 = generic fused kernel (any W%8==0, H%9==0)                   */
-    int32_t flags;          /* bit 0 (AOL_FLAG_HALO_LAST): stream a unit's 3 halo rows after its
-                               own rows instead of first (tuning experiment; same results)    */
+    int32_t flags;          /* AOL_FLAG_* bits (tuning experiments; results are identical)    */
 } aol_launch_opts_t;
 
-#define AOL_FLAG_HALO_LAST 1
+#define AOL_FLAG_HALO_LAST 1           /* stream a unit's 3 halo rows after its own rows, not first */
+#define AOL_FLAG_EVICT_FIRST_LOADS 2   /* TMA input loads with the L2 evict_first policy            */
+#define AOL_FLAG_EVICT_FIRST_STORES 4  /* TMA output stores with the L2 evict_first policy          */
 
 /* The launch configuration aol_downscale_frame_ex would use (for reports/tests). */
 typedef struct {

@@ -9,7 +9,9 @@ import ctypes
 import os
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
-LIB_PATH = os.path.join(_HERE, "libaol.so")
+# AOL_LIB_PATH lets tools load an instrumented build of the SAME library (e.g. tools/stream_probe.sh);
+# it is never a fallback: the path must hold a libaol.so built from csrc/.
+LIB_PATH = os.environ.get("AOL_LIB_PATH") or os.path.join(_HERE, "libaol.so")
 
 MAX_RANK = 8
 

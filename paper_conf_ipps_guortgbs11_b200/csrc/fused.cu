@@ -211,6 +211,8 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
     a.out_bytes = uint32_t(16 * Wo);
     a.n_consumer = plan.block - 32;
     a.halo_last = (plan.flags & AOL_FLAG_HALO_LAST) ? 1 : 0;
+    a.hint_loads = (plan.flags & AOL_FLAG_EVICT_FIRST_LOADS) ? 1 : 0;
+    a.hint_stores = (plan.flags & AOL_FLAG_EVICT_FIRST_STORES) ? 1 : 0;
 
     KernelFn k = pick(in_dtype, d_cs != nullptr, plan.block, plan.ctas_per_sm);
     aol_status_t st_attr = kernel_smem(reinterpret_cast<const void*>(k), plan.smem);

@@ -88,6 +88,8 @@ struct FusedArgs {
     uint32_t out_bytes;     // 16*Wo  (4 output rows)
     int32_t n_consumer;     // consumer threads, multiple of 32
     int32_t halo_last;      // 1: stream the halo triple after the unit's own rows
+    int32_t hint_loads;     // 1: TMA loads with L2 evict_first (input is streamed once)
+    int32_t hint_stores;    // 1: bulk stores with L2 evict_first
 };
 
 // Byte offset of 16-byte chunk `chunk` (0..7) of 128-byte line `line` under SWIZZLE_128B
@@ -184,7 +186,11 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
                     ptx::mbar_arrive_expect_tx(&full[s], a.stage_bytes);
                     uint8_t* dst = stage_base + size_t(s) * a.stage_stride;
                     if constexpr (kI32) {
-                        ptx::tma_load_3d(dst, &tmap, &full[s], 0, 0, int32_t(row0 + 3 * trip));
+                        if (a.hint_loads)
+                            ptx::tma_load_3d_hint(dst, &tmap, &full[s], 0, 0, int32_t(row0 + 3 * trip),
+                                                  ptx::policy_evict_first());
+                        else
+                            ptx::tma_load_3d(dst, &tmap, &full[s], 0, 0, int32_t(row0 + 3 * trip));
                     } else {
                         const uint8_t* src = static_cast<const uint8_t*>(a.X) + size_t(row0 + 3 * trip) * a.W;
                         ptx::bulk_load(dst, src, a.stage_bytes, &full[s]);
@@ -263,7 +269,11 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
             ptx::named_bar_sync(1, NC);
             if (tid == 0) {
                 int32_t* gz = a.Z + (size_t(plane) * a.Ho + size_t(4 * band)) * size_t(Wo);
-                ptx::bulk_store(gz, outbuf + (emit_idx % kOutBufs) * (a.out_bytes / 4), a.out_bytes);   // 4 rows
+                if (a.hint_stores)
+                    ptx::bulk_store_hint(gz, outbuf + (emit_idx % kOutBufs) * (a.out_bytes / 4), a.out_bytes,
+                                         ptx::policy_evict_first());
+                else
+                    ptx::bulk_store(gz, outbuf + (emit_idx % kOutBufs) * (a.out_bytes / 4), a.out_bytes);   // 4 rows
                 ptx::bulk_commit();
             }
             ++emit_idx;
@@ -288,7 +298,15 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
             // ---- H stage on the 3 rows of this triple: y[row][col]
             int32_t y[3][3];
 #pragma unroll
-            for (int rr = 0; rr < 3; ++rr) h_row<Tin>(sb, uint32_t(rr), g, segs, Wu, y[rr][0], y[rr][1], y[rr][2]);
+            for (int rr = 0; rr < 3; ++rr) {
+#ifdef AOL_PROBE_STREAM_ONLY
+                // measurement build only (tools/stream_probe.sh): skip the smem reads and H arithmetic to
+                // expose the pure TMA streaming rate of this access pattern.  Never in libaol.so.
+                y[rr][0] = y[rr][1] = y[rr][2] = int32_t(sb) + rr;
+#else
+                h_row<Tin>(sb, uint32_t(rr), g, segs, Wu, y[rr][0], y[rr][1], y[rr][2]);
+#endif
+            }
             __syncwarp();
             if (lane == 0) ptx::mbar_arrive(&empty[s]);
             if (++s == a.stages) {
@@ -438,6 +456,7 @@ KernelFn tma_kernel_u8(bool checksum, int block, int cps);
 template <typename Tin, bool kChecksum>
 KernelFn pick_tma_kernel(int block, int cps) {
     if (block <= 128 && cps >= 3) return fused_tma_kernel<Tin, kChecksum, 128, 4>;
+    if (block <= 320 && cps >= 3) return fused_tma_kernel<Tin, kChecksum, 320, 3>;
     if (block <= 320 && cps >= 2) return fused_tma_kernel<Tin, kChecksum, 320, 2>;
     if (block <= 512) return fused_tma_kernel<Tin, kChecksum, 512, 1>;
     return fused_tma_kernel<Tin, kChecksum, 1024, 1>;
