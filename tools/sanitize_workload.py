@@ -15,14 +15,23 @@ import paper_conf_ipps_guortgbs11_b200 as aol  # noqa: E402
 
 
 def main():
+    import argparse
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--dtypes", default="i32,u8")
+    ap.add_argument("--kernels", default="1,2")
+    ap.add_argument("--fused-only", action="store_true")
+    args = ap.parse_args()
+    dts = [{"i32": torch.int32, "u8": torch.uint8}[d] for d in args.dtypes.split(",")]
+    kernels = [int(k) for k in args.kernels.split(",")]
     torch.cuda.set_device(0)
     ok = True
     for (N, C, H, W) in [(2, 3, 27, 64), (1, 1, 9, 32), (1, 2, 18, 352)]:
-        for dt in (torch.int32, torch.uint8):
+        for dt in dts:
             x = aol.synth_frames(1, 0, N, C, H, W, "uniform", dtype=dt)
             ref = None
-            for opts in ({"kernel": 2}, {"kernel": 1}, {"kernel": 1, "stages": 2, "bands_per_unit": 1},
-                         {"kernel": 1, "ctas_per_sm": 2}, {"kernel": 1, "flags": 1}):
+            all_opts = [{"kernel": 2}, {"kernel": 1}, {"kernel": 1, "stages": 2, "bands_per_unit": 1},
+                        {"kernel": 1, "ctas_per_sm": 2}, {"kernel": 1, "flags": 1}]
+            for opts in [o for o in all_opts if o["kernel"] in kernels]:
                 try:
                     z, cs = aol.downscale_frame(x, checksums=True, opts=opts)
                 except aol.AolError:
@@ -32,6 +41,8 @@ def main():
                     ref = (z.clone(), cs.clone())
                 else:
                     ok &= torch.equal(z, ref[0]) and torch.equal(cs.view(torch.int64), ref[1].view(torch.int64))
+        if args.fused_only:
+            continue
         x = aol.synth_frames(2, 0, N, C, H, W, "signed")
         y = aol.downscale_h(x)
         z = aol.downscale_v(y)
@@ -39,6 +50,10 @@ def main():
         ok &= torch.equal(z, zf)
         ok &= torch.equal(aol.frame_checksum(z).view(torch.int64),
                           aol.downscale_frame(x, checksums=True)[1].view(torch.int64))
+    if args.fused_only:
+        torch.cuda.synchronize()
+        print("sanitize workload:", "OK" if ok else "MISMATCH")
+        return 0 if ok else 1
     t = aol.make_tiler([16, 24], [2, 3], [8, 8], [0, 0], [[8, 0], [0, 8]], [[1, 0], [0, 1]])
     A = torch.arange(16 * 24, dtype=torch.int32, device="cuda").reshape(16, 24)
     G = aol.tiler_gather(t, A)
