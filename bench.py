@@ -49,6 +49,10 @@ def parse():
     p.add_argument("--seed", type=int, default=0)
     p.add_argument("--dtype", choices=["i32", "u8"], default="i32")
     p.add_argument("--opts", type=str, default="", help='launch options JSON, e.g. {"ctas_per_sm":2}')
+    p.add_argument("--stream-frames", type=int, default=0,
+                   help="configs[4] mode: a stream of this many frames, frame-sharded across the ranks (strong "
+                        "scaling), each rank cycling through a device pool of --pool unique frames")
+    p.add_argument("--pool", type=int, default=256)
     p.add_argument("--e2e-steps", type=int, default=3)
     p.add_argument("--no-e2e", action="store_true")
     p.add_argument("--no-cpu-baseline", action="store_true")
@@ -56,6 +60,9 @@ def parse():
 
 
 def workload_name(a):
+    if a.stream_frames:
+        return (f"{a.stream_frames}-frame {a.W}x{a.H} {a.channels}-channel synthetic stream frame-sharded across "
+                f"the GPUs (device pool of {a.pool} unique frames per GPU), fused h+v downscale")
     return f"{a.frames}-frame {a.W}x{a.H} {a.channels}-channel synthetic stream per GPU, fused h+v downscale"
 
 
@@ -243,7 +250,16 @@ def main():
     opts = json.loads(a.opts) if a.opts else None
 
     F, C, H, W = a.frames, a.channels, a.H, a.W
-    frame0, F = shard.weak_range(rank, world, F)
+    if a.stream_frames:
+        # configs[4]: strong scaling; this rank's frames of the global stream, processed in launches over a
+        # device pool (stream frame n of the rank uses pool slot n mod pool)
+        frame0, count = shard.strong_range(rank, world, a.stream_frames)
+        F = max(1, min(a.pool, count))
+        calls = [min(F, count - k) for k in range(0, count, F)]
+        a.no_e2e = True
+    else:
+        frame0, F = shard.weak_range(rank, world, F)
+        count, calls = F, [F]
     tdtype = torch.int32 if a.dtype == "i32" else torch.uint8
     x = aol.synth_frames(a.seed, frame0, F, C, H, W, "uniform", dtype=tdtype, device=dev)
     z = torch.empty((F, C, 4 * (H // 9), 3 * (W // 8)), dtype=torch.int32, device=dev)
@@ -251,12 +267,20 @@ def main():
     plan = aol.downscale_frame_plan(F, C, H, W, dtype=tdtype, opts=opts)
     stream = torch.cuda.current_stream(dev)
 
+    def step(record=None):
+        for j, n in enumerate(calls):
+            if record is not None:
+                record[0][j].record(stream)
+            aol.downscale_frame(x[:n], out=z[:n], checksums=cs[:n], opts=opts)
+            if record is not None:
+                record[1][j].record(stream)
+
     for _ in range(a.warmup):
-        aol.downscale_frame(x, out=z, checksums=cs, opts=opts)
+        step()
     torch.cuda.synchronize(dev)
 
-    starts = [torch.cuda.Event(enable_timing=True) for _ in range(a.steps)]
-    ends = [torch.cuda.Event(enable_timing=True) for _ in range(a.steps)]
+    starts = [[torch.cuda.Event(enable_timing=True) for _ in calls] for _ in range(a.steps)]
+    ends = [[torch.cuda.Event(enable_timing=True) for _ in calls] for _ in range(a.steps)]
     t_begin = torch.cuda.Event(enable_timing=True)
     t_end = torch.cuda.Event(enable_timing=True)
     if world > 1:
@@ -265,18 +289,19 @@ def main():
     with ClockSampler(gpu) as clk:
         t_begin.record(stream)
         for i in range(a.steps):
-            starts[i].record(stream)
-            aol.downscale_frame(x, out=z, checksums=cs, opts=opts)
-            ends[i].record(stream)
+            step((starts[i], ends[i]))
         t_end.record(stream)
         torch.cuda.synchronize(dev)
     if world > 1:
         dist.barrier()
     elapsed_ms = t_begin.elapsed_time(t_end)
-    launch_ms = [s.elapsed_time(e) for s, e in zip(starts, ends)]
+    launch_ms = [s.elapsed_time(e) for ss, es in zip(starts, ends) for s, e in zip(ss, es)]
+    launch_frames = [n for _ in range(a.steps) for n in calls]
 
     # max over ranks (NCCL), and gather per-rank checksums: the only cross-GPU traffic
-    max_ms, cs_all_t = shard.gather_results(cs if backend == "nccl" else cs.cpu(), elapsed_ms)
+    counts = ([max(1, min(a.pool, shard.strong_range(r, world, a.stream_frames)[1])) for r in range(world)]
+              if a.stream_frames else None)
+    max_ms, cs_all_t = shard.gather_results(cs if backend == "nccl" else cs.cpu(), elapsed_ms, counts=counts)
     cs_all = cs_all_t.cpu().numpy().view(np.uint64) if world > 1 else None
 
     # e2e through the host-buffer C-ABI call
@@ -312,26 +337,30 @@ def main():
             dist.destroy_process_group()
         return
 
-    value = world * F * a.steps / (max_ms / 1000.0)
+    total_frames = (a.stream_frames if a.stream_frames else world * F) * a.steps
+    value = total_frames / (max_ms / 1000.0)
     bpf = bytes_per_frame(a)
     avg_launch_s = statistics.mean(launch_ms) / 1000.0
-    achieved = bpf * F / avg_launch_s / 1e9
+    # algorithmic bytes over kernel time, summed over this rank's launches (all equal in the default mode)
+    achieved = bpf * sum(launch_frames) / (sum(launch_ms) / 1000.0) / 1e9
     peak, peak_src = measured_peak()
     traffic = ncu_traffic(a)
     line = {
         "metric": METRIC, "value": value, "unit": "frames/s", "n_gpus": world, "steps": a.steps,
-        "warmup": a.warmup, "ms_per_step": max_ms / a.steps, "higher_is_better": True, "scaling": "weak",
+        "warmup": a.warmup, "ms_per_step": max_ms / a.steps, "higher_is_better": True,
+        "scaling": "strong" if a.stream_frames else "weak",
         "vs_baseline": None, "dtype": a.dtype, "data": "synthetic",
-        "config": {"workload": workload_name(a), "frames_per_gpu": F, "H": H, "W": W, "channels": C,
+        "config": {"workload": workload_name(a), "frames_per_gpu": count, "launches_per_step": len(calls),
+                   "H": H, "W": W, "channels": C,
                    "in_dtype": a.dtype, "out_dtype": "i32", "l2": "inputs (7.46 GB at HD int32) larger than L2; no flush",
                    "parallelism": f"frame-sharded x{world} (no data-path collective)",
                    "kernel": {"1": "fused_tma_kernel", "2": "fused_generic_kernel"}[str(plan["kernel"])],
                    "plan": plan},
         "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s", "frac": achieved / peak,
                      "traffic": traffic, "peak_source": peak_src,
-                     "algorithmic_bytes_per_launch": bpf * F,
+                     "algorithmic_bytes_per_launch": bpf * calls[0],
                      "avg_launch_ms": avg_launch_s * 1000.0, "min_launch_ms": min(launch_ms)},
-        "gpu_launches": a.steps,
+        "gpu_launches": a.steps * len(calls),
         "clocks": clk.summary(),
     }
     if e2e is not None:

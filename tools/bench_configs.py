@@ -178,6 +178,15 @@ def main():
               "equals_fused": bool(torch.equal(zf.reshape(N * C, 480, 720), z))})
         del x, y, z, zf
         torch.cuda.empty_cache()
+    if want("d5"):
+        # configs[4] on one GPU: the 10,000-frame stream through bench.py's strong-scaling mode
+        import subprocess
+        r = subprocess.run([sys.executable, os.path.join(ROOT, "bench.py"), "--stream-frames", "10000", "--pool", "256",
+                            "--steps", "5", "--warmup", "2", "--no-cpu-baseline"], capture_output=True, text=True)
+        line = json.loads(r.stdout.strip().splitlines()[-1])
+        emit({"config": "d5 10,000-frame HD stream, 1 GPU (pool 256)", "frames_per_s": line["value"],
+              "ms_per_step": line["ms_per_step"], "GBps": line["roofline"]["achieved"],
+              "launches_per_step": line["config"]["launches_per_step"], "scaling": line["scaling"]})
     if want("d4"):
         fused_line("d4 4K batch", 64, 3, 2160, 3840)
     if want("f1"):
