@@ -104,7 +104,7 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, const void* d_in, const int32_t* d
     }
     if (o.kernel == 1 && !tma_ok) {
         set_error("TMA fused kernel requested but unsupported for this shape/dtype/alignment "
-                  "(int32: W %% 32 == 0, W <= 7936; uint8: W %% 16 == 0; 16-byte aligned buffers)");
+                  "(int32: W %% 32 == 0 and W <= 7680; uint8: W %% 16 == 0 and W <= 7936; 16-byte aligned buffers)");
         return AOL_E_SHAPE;
     }
     if (o.kernel == 2) tma_ok = false;

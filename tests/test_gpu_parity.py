@@ -356,3 +356,64 @@ def test_host_streamed_matches_device(orc):
     zo, cso = run_oracle(orc, xh)
     assert np.array_equal(zh.numpy(), zo)
     assert np.array_equal(csh.view(torch.int64).numpy().view(np.uint64), cso)
+
+
+# -------------------------------------------------------------- edge cases
+
+@pytest.mark.parametrize("W,dtype,kernel", [(7680, torch.int32, 1), (7936, torch.int32, 2), (7936, torch.uint8, 1),
+                                            (8192, torch.uint8, 2), (16, torch.uint8, 1), (32, torch.int32, 1)])
+def test_width_limits(orc, W, dtype, kernel):
+    """Widest frames the TMA kernel takes and the first widths that fall back to the generic kernel: int32
+    needs two 3-row stages + one 4-row output band in 227 KB of smem (W <= 7680); uint8 is capped by
+    W/8 <= 992 consumer threads + 1 producer warp = 1024.  Also the narrowest TMA widths."""
+    N, C, H = 1, 1, 18
+    xh = synth.frames(61, 0, N, C, H, W, "uniform")
+    zo, cso = run_oracle(orc, xh)
+    x = torch.from_numpy(xh.astype(np.uint8) if dtype == torch.uint8 else xh).cuda()
+    assert aol.downscale_frame_plan(N, C, H, W, dtype=dtype)["kernel"] == kernel
+    z, cs = aol.downscale_frame(x, checksums=True)
+    torch.cuda.synchronize()
+    assert np.array_equal(z.cpu().numpy(), zo)
+    assert np.array_equal(np_u64(cs), cso)
+
+
+def test_misaligned_and_noncontiguous_inputs():
+    base = torch.zeros(1 * 3 * 18 * 64 + 4, dtype=torch.int32, device="cuda")
+    x = base[1:1 + 3 * 18 * 64].view(1, 3, 18, 64)          # 4-byte offset: not 16-byte aligned
+    with pytest.raises(aol.AolError) as e:
+        aol.downscale_frame(x)
+    assert e.value.status == aol._lib.E_ALIGN
+    y = torch.zeros((1, 3, 18, 128), dtype=torch.int32, device="cuda")[..., ::2]
+    with pytest.raises(ValueError):
+        aol.downscale_frame(y)
+
+
+def test_concurrent_streams_and_threads(orc):
+    """The library is re-entrant: four host threads, four streams, interleaved launches."""
+    import threading
+
+    shapes = [(3, 3, 36, 256), (2, 3, 288, 352), (4, 1, 27, 1920), (2, 2, 18, 512)]
+    inputs = [synth.frames(70 + i, 0, *s) for i, s in enumerate(shapes)]
+    results, errors = [None] * 4, []
+
+    def work(i):
+        try:
+            s = torch.cuda.Stream()
+            with torch.cuda.stream(s):
+                x = torch.from_numpy(inputs[i]).cuda()
+                for _ in range(5):
+                    z, cs = aol.downscale_frame(x, checksums=True, stream=s)
+                s.synchronize()
+                results[i] = (z.cpu().numpy(), np_u64(cs))
+        except Exception as e:  # pragma: no cover - reported below
+            errors.append(e)
+
+    ts = [threading.Thread(target=work, args=(i,)) for i in range(4)]
+    for t in ts:
+        t.start()
+    for t in ts:
+        t.join()
+    assert not errors, errors
+    for i in range(4):
+        zo, cso = run_oracle(orc, inputs[i])
+        assert np.array_equal(results[i][0], zo) and np.array_equal(results[i][1], cso)
