@@ -110,6 +110,8 @@ typedef struct {
 #define AOL_FLAG_HALO_LAST 1           /* stream a unit's 3 halo rows after its own rows, not first */
 #define AOL_FLAG_EVICT_FIRST_LOADS 2   /* TMA input loads with the L2 evict_first policy            */
 #define AOL_FLAG_EVICT_FIRST_STORES 4  /* TMA output stores with the L2 evict_first policy          */
+#define AOL_FLAG_BLOCKED_UNITS 8       /* each CTA takes a contiguous block of work units (default:
+                                          round-robin, so concurrently running CTAs are adjacent)  */
 
 /* The launch configuration aol_downscale_frame_ex would use (for reports/tests). */
 typedef struct {

@@ -39,8 +39,10 @@ aol_status_t get_encode_fn(EncodeTiledFn* fn) {
     return AOL_OK;
 }
 
-bool tma_shape_ok(aol_dtype_t dt, int64_t planes, int64_t H, int64_t W) {
+bool tma_shape_ok(aol_dtype_t dt, int64_t planes, int64_t channels, int64_t H, int64_t W) {
     if (H < 9 || W / 8 > kMaxConsumers) return false;
+    // checksum weights (1 + frame-local output index) are computed in 32 bits
+    if (channels * (4 * (H / 9)) * (3 * (W / 8)) >= (int64_t(1) << 32) - 1) return false;
     if (dt == AOL_I32) return W % 32 == 0 && W / 32 <= 256 && planes * H < (int64_t(1) << 31);
     if (dt == AOL_U8) return W % 16 == 0;   // 1-D bulk copies: 16-byte granularity
     return false;
@@ -63,7 +65,7 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, const void* d_in, const int32_t* d
     *plan = FusedPlan{};
     plan->num_sms = dev.num_sms;
 
-    bool tma_ok = tma_shape_ok(in_dtype, planes, H, W) && (d_in == nullptr || aligned16(d_in)) &&
+    bool tma_ok = tma_shape_ok(in_dtype, planes, channels, H, W) && (d_in == nullptr || aligned16(d_in)) &&
                   (d_out == nullptr || aligned16(d_out));
     const int es = in_dtype == AOL_U8 ? 1 : 4;
     const uint32_t stage_bytes = uint32_t(3 * W * es);
@@ -213,6 +215,7 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
     a.halo_last = (plan.flags & AOL_FLAG_HALO_LAST) ? 1 : 0;
     a.hint_loads = (plan.flags & AOL_FLAG_EVICT_FIRST_LOADS) ? 1 : 0;
     a.hint_stores = (plan.flags & AOL_FLAG_EVICT_FIRST_STORES) ? 1 : 0;
+    a.blocked_units = (plan.flags & AOL_FLAG_BLOCKED_UNITS) ? 1 : 0;
 
     KernelFn k = pick(in_dtype, d_cs != nullptr, plan.block, plan.ctas_per_sm);
     aol_status_t st_attr = kernel_smem(reinterpret_cast<const void*>(k), plan.smem);

@@ -90,12 +90,21 @@ struct FusedArgs {
     int32_t halo_last;      // 1: stream the halo triple after the unit's own rows
     int32_t hint_loads;     // 1: TMA loads with L2 evict_first (input is streamed once)
     int32_t hint_stores;    // 1: bulk stores with L2 evict_first
+    int32_t blocked_units;  // 1: contiguous block of units per CTA instead of round-robin
 };
 
 // Byte offset of 16-byte chunk `chunk` (0..7) of 128-byte line `line` under SWIZZLE_128B
 // (chunk index XOR line index mod 8; stage buffers are 1024-byte aligned).
 __device__ __forceinline__ uint32_t swz(uint32_t line, uint32_t chunk) {
     return (line << 7) | (((chunk ^ line) & 7u) << 4);
+}
+
+// k-th work unit of this CTA: round-robin (concurrently running CTAs stream adjacent units) or, with
+// AOL_FLAG_BLOCKED_UNITS, a contiguous block of units per CTA.  Returns >= nunits when done.
+__device__ __forceinline__ int64_t unit_of(const FusedArgs& a, int64_t k) {
+    if (!a.blocked_units) return int64_t(blockIdx.x) + k * gridDim.x;
+    const int64_t per = (a.nunits + gridDim.x - 1) / gridDim.x;
+    return k < per ? int64_t(blockIdx.x) * per + k : a.nunits;
 }
 
 // Per-thread constants of the H stage (which repetition, where its bytes live).
@@ -171,7 +180,7 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
             if (kI32) ptx::prefetch_tensormap(&tmap);
             int s = 0;
             uint32_t ph = 0;
-            for (int64_t u = blockIdx.x; u < a.nunits; u += gridDim.x) {
+            for (int64_t k = 0, u = unit_of(a, 0); u < a.nunits; u = unit_of(a, ++k)) {
                 const int64_t plane = u / a.units_per_plane;
                 const int32_t b0 = int32_t(u - plane * a.units_per_plane) * a.bands_per_unit;
                 const int32_t b1 = min(b0 + a.bands_per_unit, a.nbands);
@@ -233,7 +242,7 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
     uint32_t ph = 0;
     uint32_t emit_idx = 0;
 
-    for (int64_t u = blockIdx.x; u < a.nunits; u += gridDim.x) {
+    for (int64_t k = 0, u = unit_of(a, 0); u < a.nunits; u = unit_of(a, ++k)) {
         const int64_t plane = u / a.units_per_plane;
         const int32_t b0 = int32_t(u - plane * a.units_per_plane) * a.bands_per_unit;
         const int32_t b1 = min(b0 + a.bands_per_unit, a.nbands);
@@ -278,13 +287,15 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
             }
             ++emit_idx;
             if (kChecksum && active) {
-                const uint64_t w0 =
-                    1u + (uint64_t(chan) * a.Ho + uint64_t(4 * band)) * uint64_t(Wo) + uint64_t(3 * r);
+                // weight = 1 + frame-local flat index < 2^32 (the planner guarantees C*Ho*Wo < 2^32), so each
+                // term is one 32x32->64 multiply-add (IMAD.WIDE.U32 with a 64-bit addend)
+                const uint32_t w0 = 1u + (uint32_t(chan) * uint32_t(a.Ho) + uint32_t(4 * band)) * uint32_t(Wo) +
+                                    uint32_t(3 * r);
 #pragma unroll
                 for (int k = 0; k < 4; ++k)
 #pragma unroll
                     for (int m = 0; m < 3; ++m)
-                        csacc += uint64_t(uint32_t(z[k][m])) * (w0 + uint64_t(k) * Wo + uint64_t(m));
+                        csacc += uint64_t(uint32_t(z[k][m])) * uint64_t(w0 + uint32_t(k * Wo + m));
             }
         };
 
