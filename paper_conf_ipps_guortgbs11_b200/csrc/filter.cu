@@ -8,13 +8,16 @@
 //
 // Per repetition r (one thread): base coordinates of both tilers are o' + P'.r reduced mod
 // the extents once; the pattern-element and output-element offsets F'.i are host-precomputed
-// tables already reduced mod the extents, so every element costs an add, a conditional
-// subtract and an FMA per array dimension.
+// tables already reduced mod the extents.  A repetition whose whole pattern stays inside the
+// array (every repetition of a non-wrapping tiler; all but the last repetition of a row for the
+// paper's H tiler) takes the fast path: element = base + lin[p], one add per element.  The
+// others apply the toroidal wrap per dimension (add, conditional subtract, FMA).
 #include <cuda_runtime.h>
 
 #include <algorithm>
 #include <cstdint>
 #include <cstring>
+#include <type_traits>
 
 #include "common.h"
 
@@ -34,18 +37,23 @@ struct FilterDev {
     int32_t start[AOL_MAX_WINDOWS];
     int32_t f_in[AOL_MAX_FILTER_PATTERN][AOL_MAX_RANK];  // F'.i(p) mod s, per input pattern element
     int32_t f_out[AOL_MAX_WINDOWS][AOL_MAX_RANK];        // F'.i(k) mod s, per output element
+    // fast path: a repetition whose reference point + the largest pattern coordinate stays inside every
+    // extent needs no modulo, and its elements sit at base + lin[p] (row-major element offsets)
+    int32_t fmax_in[AOL_MAX_RANK], fmax_out[AOL_MAX_RANK];
+    int64_t lin_in[AOL_MAX_FILTER_PATTERN], lin_out[AOL_MAX_WINDOWS];
 };
 
-template <bool kFast32>
+// D bounds every rank involved (array ranks of both tilers, repetition rank): loops unroll to D.
+template <int D, bool kFast32>
 __global__ void __launch_bounds__(256) filter_kernel(const FilterDev fd, const int32_t* __restrict__ in,
                                                      int32_t* __restrict__ out) {
     for (int64_t r = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; r < fd.nrep;
          r += int64_t(gridDim.x) * blockDim.x) {
         // repetition multi-index (last dim fastest)
-        int64_t ridx[AOL_MAX_RANK];
+        int64_t ridx[D];
         int64_t g = r;
 #pragma unroll
-        for (int j = AOL_MAX_RANK - 1; j >= 0; --j) {
+        for (int j = D - 1; j >= 0; --j) {
             if (j < fd.rr) {
                 if (kFast32) {
                     const uint32_t n = uint32_t(g);
@@ -62,12 +70,12 @@ __global__ void __launch_bounds__(256) filter_kernel(const FilterDev fd, const i
             }
         }
         // reference points o' + P'.r  (mod s), Section IV
-        int32_t bin[AOL_MAX_RANK], bout[AOL_MAX_RANK];
+        int32_t bin[D], bout[D];
 #pragma unroll
-        for (int a = 0; a < AOL_MAX_RANK; ++a) {
+        for (int a = 0; a < D; ++a) {
             int64_t vi = fd.o_in[a], vo = fd.o_out[a];
 #pragma unroll
-            for (int j = 0; j < AOL_MAX_RANK; ++j) {
+            for (int j = 0; j < D; ++j) {
                 if (j < fd.rr) {
                     vi += int64_t(fd.P_in[a][j]) * ridx[j];
                     vo += int64_t(fd.P_out[a][j]) * ridx[j];
@@ -76,30 +84,51 @@ __global__ void __launch_bounds__(256) filter_kernel(const FilterDev fd, const i
             bin[a] = a < fd.ra_in ? int32_t(vi % fd.s_in[a]) : 0;
             bout[a] = a < fd.ra_out ? int32_t(vo % fd.s_out[a]) : 0;
         }
+        bool in_ok = true, out_ok = true;
+        int64_t base_in = 0, base_out = 0;
+#pragma unroll
+        for (int a = 0; a < D; ++a) {
+            if (a < fd.ra_in) {
+                in_ok &= bin[a] + fd.fmax_in[a] < fd.s_in[a];
+                base_in += int64_t(bin[a]) * fd.st_in[a];
+            }
+            if (a < fd.ra_out) {
+                out_ok &= bout[a] + fd.fmax_out[a] < fd.s_out[a];
+                base_out += int64_t(bout[a]) * fd.st_out[a];
+            }
+        }
+        const int32_t* inb = in + base_in;
         for (int k = 0; k < fd.n_win; ++k) {
             // task (Fig. 5): S over the window, tile = S/d - S%d
             int32_t S = 0;
-            for (int t = 0; t < fd.len; ++t) {
-                const int p = fd.start[k] + t;
-                int64_t off = 0;
+            if (in_ok) {
+                for (int t = 0; t < fd.len; ++t) S += __ldg(inb + fd.lin_in[fd.start[k] + t]);
+            } else {
+                for (int t = 0; t < fd.len; ++t) {
+                    const int p = fd.start[k] + t;
+                    int64_t off = 0;
 #pragma unroll
-                for (int a = 0; a < AOL_MAX_RANK; ++a) {
-                    if (a < fd.ra_in) {
-                        int32_t c = bin[a] + fd.f_in[p][a];   // pattern element
-                        if (c >= fd.s_in[a]) c -= fd.s_in[a];
-                        off += int64_t(c) * fd.st_in[a];
+                    for (int a = 0; a < D; ++a) {
+                        if (a < fd.ra_in) {
+                            int32_t c = bin[a] + fd.f_in[p][a];   // pattern element, toroidal
+                            if (c >= fd.s_in[a]) c -= fd.s_in[a];
+                            off += int64_t(c) * fd.st_in[a];
+                        }
                     }
+                    S += __ldg(in + off);
                 }
-                S += __ldg(in + off);
             }
             const int32_t tile = S / fd.divisor - S % fd.divisor;
-            int64_t off = 0;
+            int64_t off = base_out + fd.lin_out[k];
+            if (!out_ok) {
+                off = 0;
 #pragma unroll
-            for (int a = 0; a < AOL_MAX_RANK; ++a) {
-                if (a < fd.ra_out) {
-                    int32_t c = bout[a] + fd.f_out[k][a];       // output tiler (Fig. 6)
-                    if (c >= fd.s_out[a]) c -= fd.s_out[a];
-                    off += int64_t(c) * fd.st_out[a];
+                for (int a = 0; a < D; ++a) {
+                    if (a < fd.ra_out) {
+                        int32_t c = bout[a] + fd.f_out[k][a];       // output tiler (Fig. 6), toroidal
+                        if (c >= fd.s_out[a]) c -= fd.s_out[a];
+                        off += int64_t(c) * fd.st_out[a];
+                    }
                 }
             }
             out[off] = tile;
@@ -271,15 +300,29 @@ aol_status_t aol_filter_apply(const aol_filter_t* f, const int32_t* d_in, int32_
     for (int k = 0; k < fd.n_win; ++k) fd.start[k] = f->window_start[k];
     fill_offsets(&f->in, fd.n_in, fd.f_in);
     fill_offsets(&f->out, fd.n_win, fd.f_out);
+    for (int a = 0; a < AOL_MAX_RANK; ++a) {
+        for (int p = 0; p < fd.n_in; ++p) fd.fmax_in[a] = std::max(fd.fmax_in[a], fd.f_in[p][a]);
+        for (int k = 0; k < fd.n_win; ++k) fd.fmax_out[a] = std::max(fd.fmax_out[a], fd.f_out[k][a]);
+    }
+    for (int p = 0; p < fd.n_in; ++p)
+        for (int a = 0; a < fd.ra_in; ++a) fd.lin_in[p] += int64_t(fd.f_in[p][a]) * fd.st_in[a];
+    for (int k = 0; k < fd.n_win; ++k)
+        for (int a = 0; a < fd.ra_out; ++a) fd.lin_out[k] += int64_t(fd.f_out[k][a]) * fd.st_out[a];
 
     DeviceInfo dev;
     st = device_info(&dev);
     if (st != AOL_OK) return st;
     const int grid = int(std::max<int64_t>(1, std::min<int64_t>((fd.nrep + 255) / 256, int64_t(dev.num_sms) * 16)));
-    if (fd.fast32)
-        filter_kernel<true><<<grid, 256, 0, s>>>(fd, d_in, d_out);
-    else
-        filter_kernel<false><<<grid, 256, 0, s>>>(fd, d_in, d_out);
+    const int D = std::max(fd.rr, std::max(fd.ra_in, fd.ra_out));
+    auto launch = [&](auto kfast, auto kd) {
+        filter_kernel<decltype(kd)::value, decltype(kfast)::value><<<grid, 256, 0, s>>>(fd, d_in, d_out);
+    };
+    using T = std::true_type;
+    using F = std::false_type;
+    if (D <= 2) fd.fast32 ? launch(T{}, std::integral_constant<int, 2>{}) : launch(F{}, std::integral_constant<int, 2>{});
+    else if (D <= 3) fd.fast32 ? launch(T{}, std::integral_constant<int, 3>{}) : launch(F{}, std::integral_constant<int, 3>{});
+    else if (D <= 4) fd.fast32 ? launch(T{}, std::integral_constant<int, 4>{}) : launch(F{}, std::integral_constant<int, 4>{});
+    else fd.fast32 ? launch(T{}, std::integral_constant<int, 8>{}) : launch(F{}, std::integral_constant<int, 8>{});
     AOL_LAUNCH_CHECK("filter_kernel");
     return AOL_OK;
 }
