@@ -12,7 +12,9 @@ NVFLAGS   := $(ARCH) -O3 -lineinfo -std=c++17 -Xcompiler -fPIC,-fvisibility=hidd
              --expt-relaxed-constexpr
 ORACLE    := oracle/liboracle.so
 
-all: $(LIB) $(ORACLE)
+EXAMPLE   := $(BUILD)/aol_example
+
+all: $(LIB) $(ORACLE) $(EXAMPLE)
 
 $(BUILD)/%.o: $(PKG)/csrc/%.cu $(CHDR)
 	@mkdir -p $(BUILD)
@@ -21,6 +23,12 @@ $(BUILD)/%.o: $(PKG)/csrc/%.cu $(CHDR)
 $(LIB): $(OBJS)
 	$(NVCC) $(ARCH) -shared -cudart static -o $@.tmp $(OBJS) -lrt -ldl -lpthread
 	mv $@.tmp $@
+
+# a plain-C client of the C ABI (no Python): examples/aol_example.c
+$(EXAMPLE): examples/aol_example.c include/aol.h $(LIB)
+	@mkdir -p $(BUILD)
+	gcc -std=c99 -O2 -Wall -Wextra -I include -I /usr/local/cuda/include $< -L $(PKG) -laol \
+	    -L /usr/local/cuda/lib64 -lcudart -Wl,-rpath,'$$ORIGIN/../$(PKG)' -o $@
 
 $(ORACLE): oracle/aol_oracle.c oracle/aol_oracle.h
 	gcc -std=c99 -O2 -fopenmp -fPIC -shared -Wall -Wextra -o $@ oracle/aol_oracle.c

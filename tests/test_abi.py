@@ -205,3 +205,16 @@ def test_kernel_division_identities():
     assert np.array_equal(q - np.fmod(S, 6), 7 * q - S)
     U = np.arange(0, 98304, dtype=np.uint64)
     assert np.array_equal(((U * np.uint64(43691)) & np.uint64(0xFFFFFFFF)) >> np.uint64(18), U // np.uint64(6))
+
+
+def test_c_example_builds_against_header():
+    """examples/aol_example.c compiles and links against include/aol.h + libaol.so with gcc (C99)."""
+    import subprocess
+    import tempfile
+
+    out = os.path.join(tempfile.mkdtemp(), "aol_example")
+    subprocess.check_call(["gcc", "-std=c99", "-O2", "-Wall", "-Wextra", "-Werror", "-I", os.path.join(ROOT, "include"),
+                           "-I", "/usr/local/cuda/include", os.path.join(ROOT, "examples", "aol_example.c"),
+                           "-L", os.path.dirname(_lib.LIB_PATH), "-laol", "-L", "/usr/local/cuda/lib64", "-lcudart",
+                           "-o", out])
+    assert os.path.exists(out)
