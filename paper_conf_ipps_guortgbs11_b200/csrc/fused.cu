@@ -86,7 +86,7 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, const void* d_in, const int32_t* d
                                 : std::max(1, std::min(8, (want_warps + cwarps - 1) / cwarps));
         for (;; --cps) {
             const int budget = std::min(dev.smem_optin, dev.smem_per_sm / cps - 1024);
-            const int fixed = kOutBufs * int(out_bytes) + 2 * kMaxStages * 8 + 1024;  // out, barriers, slack
+            const int fixed = kOutBufs * int(out_bytes) + 2 * kMaxStages * 8 + 256 + 1024;  // out, barriers, red, slack
             stages = std::min((budget - fixed) / int(stage_stride), kMaxStages);
             if (o.stages > 0) {
                 stages = std::min(stages, o.stages);
@@ -95,7 +95,7 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, const void* d_in, const int32_t* d
                 stages = std::min(stages, std::max(2, target));
             }
             int occ = 0;
-            const int smem = stages * int(stage_stride) + kOutBufs * int(out_bytes) + 2 * stages * 8 + 1024;
+            const int smem = stages * int(stage_stride) + kOutBufs * int(out_bytes) + 2 * stages * 8 + 256 + 1024;
             if (stages >= 2 && cps > 1) occ = kernel_occupancy(reinterpret_cast<const void*>(pick(in_dtype, true, block, cps)), block, smem);
             if (cps == 1) occ = 1;   // one CTA always fits once its shared memory does
             if ((stages >= 2 && occ >= cps) || cps == 1 || o.ctas_per_sm > 0) {
@@ -137,7 +137,7 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, const void* d_in, const int32_t* d
         plan->grid = int(std::min<int64_t>(plan->units, max_ctas));
         plan->block = block;
         plan->stages = stages;
-        plan->smem = stages * int(stage_stride) + kOutBufs * int(out_bytes) + 2 * stages * 8 + 1024;
+        plan->smem = stages * int(stage_stride) + kOutBufs * int(out_bytes) + 2 * stages * 8 + 256 + 1024;
         plan->ctas_per_sm = cps;
         plan->flags = o.flags;
     } else {

@@ -1,4 +1,4 @@
-// fused.cu -- K-5: the fused HD->SD downscaler (hf -> vf of Fig. 3 in one kernel).
+// fused_kernel.cuh -- K-5: the fused HD->SD downscaler (hf -> vf of Fig. 3 in one kernel).
 //
 // What it computes: per plane X[H][W] (one colour channel)
 //   H stage  (Fig. 10 tilers P:L681-694, Fig. 5 task P:L435-446):
@@ -32,7 +32,7 @@
 //    (4 outputs x 3 columns per thread), so every input row is read once.
 //  * Each finished band (4 output rows, contiguous in Z) is staged in smem and
 //    written by one 1-D TMA bulk store; the per-frame checksum is folded in
-//    registers and added with one atomic per warp per unit.
+//    registers, reduced across the CTA and added with one atomic per unit.
 #pragma once
 #include <cuda.h>
 #include <cuda_runtime.h>
@@ -162,6 +162,7 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
     int32_t* outbuf = reinterpret_cast<int32_t*>(smem + size_t(a.stages) * a.stage_stride);
     uint64_t* full = reinterpret_cast<uint64_t*>(smem + size_t(a.stages) * a.stage_stride + kOutBufs * a.out_bytes);
     uint64_t* empty = full + a.stages;
+    unsigned long long* red = reinterpret_cast<unsigned long long*>(empty + a.stages);   // [32] checksum partials
 
     const int tid = threadIdx.x;
     const int NC = a.n_consumer;
@@ -373,11 +374,17 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
         emit(b1 - 1, Hr9, Hr911);   // the unit's last band, completed by the halo rows
 
         if (kChecksum) {
+            // warp -> CTA reduction, then ONE atomic per unit (many units of one frame hit the same address)
 #pragma unroll
             for (int off = 16; off > 0; off >>= 1) csacc += __shfl_xor_sync(0xffffffffu, csacc, off);
-            if (lane == 0 && csacc != 0)
-                atomicAdd(reinterpret_cast<unsigned long long*>(a.cs + plane / a.channels),
-                          static_cast<unsigned long long>(csacc));
+            if (lane == 0) red[tid >> 5] = csacc;
+            ptx::named_bar_sync(2, NC);
+            if (tid == 0) {
+                unsigned long long sum = 0;
+                for (int w = 0; w < NC / 32; ++w) sum += red[w];
+                atomicAdd(reinterpret_cast<unsigned long long*>(a.cs + plane / a.channels), sum);
+            }
+            ptx::named_bar_sync(2, NC);   // red[] is reused by the next unit
         }
     }
     if (tid == 0) ptx::bulk_wait<0>();
