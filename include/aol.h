@@ -112,6 +112,7 @@ typedef struct {
 #define AOL_FLAG_EVICT_FIRST_STORES 4  /* TMA output stores with the L2 evict_first policy          */
 #define AOL_FLAG_BLOCKED_UNITS 8       /* each CTA takes a contiguous block of work units (default:
                                           round-robin, so concurrently running CTAs are adjacent)  */
+#define AOL_FLAG_U8_BULK 16            /* uint8 input: 1-D bulk copies even when W % 128 == 0      */
 
 /* The launch configuration aol_downscale_frame_ex would use (for reports/tests). */
 typedef struct {

@@ -189,7 +189,26 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
             return AOL_E_CUDA;
         }
     }
+    const bool u8_tensor = in_dtype == AOL_U8 && W % 128 == 0 && W / 128 <= 256 &&
+                           planes * H < (int64_t(1) << 31) && !(plan.flags & AOL_FLAG_U8_BULK);
+    if (u8_tensor) {
+        EncodeTiledFn encode;
+        aol_status_t st = get_encode_fn(&encode);
+        if (st != AOL_OK) return st;
+        const cuuint64_t gdim[3] = {128, cuuint64_t(W / 128), cuuint64_t(planes * H)};
+        const cuuint64_t gstride[2] = {128, cuuint64_t(W)};
+        const cuuint32_t box[3] = {128, cuuint32_t(W / 128), 3};
+        const cuuint32_t estr[3] = {1, 1, 1};
+        CUresult cr = encode(&map, CU_TENSOR_MAP_DATA_TYPE_UINT8, 3, const_cast<void*>(d_in), gdim, gstride, box,
+                             estr, CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE,
+                             CU_TENSOR_MAP_L2_PROMOTION_L2_256B, CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+        if (cr != CUDA_SUCCESS) {
+            set_error("cuTensorMapEncodeTiled (uint8) failed (CUresult %d)", int(cr));
+            return AOL_E_CUDA;
+        }
+    }
     FusedArgs a;
+    a.u8_tensor = u8_tensor ? 1 : 0;
     a.Z = d_out;
     a.cs = d_cs;
     a.X = d_in;

@@ -20,8 +20,9 @@
 //    round-robin.
 //  * One producer warp fills an S-stage smem ring guarded by full/empty
 //    mbarriers.  int32 input: 3-D TMA tensor loads (box = 3 rows x W,
-//    SWIZZLE_128B).  uint8 input ("24-bit RGB"): 1-D TMA bulk copies of
-//    the contiguous 3-row triple.
+//    SWIZZLE_128B).  uint8 input ("24-bit RGB"): 3-D TMA tensor loads of
+//    {128 B, W/128, 3 rows} without swizzle when W % 128 == 0, else 1-D TMA bulk
+//    copies of the contiguous 3-row triple (same smem layout either way).
 //  * Consumer thread r owns repetition r (8 input columns -> 3 Y columns).
 //    int32: two conflict-free LDS.128 per row (the 128B swizzle spreads the
 //    32-byte per-thread stride over all banks).  uint8: one LDS.64 per row and
@@ -91,6 +92,7 @@ struct FusedArgs {
     int32_t hint_loads;     // 1: TMA loads with L2 evict_first (input is streamed once)
     int32_t hint_stores;    // 1: bulk stores with L2 evict_first
     int32_t blocked_units;  // 1: contiguous block of units per CTA instead of round-robin
+    int32_t u8_tensor;      // uint8 path: 1 = 3-D TMA tensor loads (W % 128 == 0), 0 = 1-D bulk copies
 };
 
 // Byte offset of 16-byte chunk `chunk` (0..7) of 128-byte line `line` under SWIZZLE_128B
@@ -178,7 +180,7 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
     if (tid >= NC) {
         // ------------------------------------------------ producer warp (TMA)
         if (tid == NC) {
-            if (kI32) ptx::prefetch_tensormap(&tmap);
+            if (kI32 || a.u8_tensor) ptx::prefetch_tensormap(&tmap);
             int s = 0;
             uint32_t ph = 0;
             for (int64_t k = 0, u = unit_of(a, 0); u < a.nunits; u = unit_of(a, ++k)) {
@@ -201,6 +203,9 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
                                                   ptx::policy_evict_first());
                         else
                             ptx::tma_load_3d(dst, &tmap, &full[s], 0, 0, int32_t(row0 + 3 * trip));
+                    } else if (a.u8_tensor) {
+                        // {128 B, W/128, rows} tensor, no swizzle: same linear smem layout as the bulk copy
+                        ptx::tma_load_3d(dst, &tmap, &full[s], 0, 0, int32_t(row0 + 3 * trip));
                     } else {
                         const uint8_t* src = static_cast<const uint8_t*>(a.X) + size_t(row0 + 3 * trip) * a.W;
                         ptx::bulk_load(dst, src, a.stage_bytes, &full[s]);

@@ -20,12 +20,16 @@ def main():
     ap.add_argument("--dtypes", default="i32,u8")
     ap.add_argument("--kernels", default="1,2")
     ap.add_argument("--fused-only", action="store_true")
+    ap.add_argument("--widths", default="", help="only these W values, e.g. 256")
     args = ap.parse_args()
     dts = [{"i32": torch.int32, "u8": torch.uint8}[d] for d in args.dtypes.split(",")]
     kernels = [int(k) for k in args.kernels.split(",")]
     torch.cuda.set_device(0)
     ok = True
-    for (N, C, H, W) in [(2, 3, 27, 64), (1, 1, 9, 32), (1, 2, 18, 352)]:
+    shapes = [(2, 3, 27, 64), (1, 1, 9, 32), (1, 2, 18, 352), (2, 2, 18, 256)]
+    if args.widths:
+        shapes = [sh for sh in shapes if str(sh[3]) in args.widths.split(",")]
+    for (N, C, H, W) in shapes:
         for dt in dts:
             x = aol.synth_frames(1, 0, N, C, H, W, "uniform", dtype=dt)
             ref = None
