@@ -258,6 +258,9 @@ def test_filter_presets_vs_oracle(orc, shape):
     z = aol.filter_apply(aol.filter_preset(aol.FILTER_V, P, H, 3 * W // 8), y)
     torch.cuda.synchronize()
     assert np.array_equal(z.cpu().numpy(), orc.downscale_v(yo))
+    # cross-path: generic run-time repetitions == the specialised fused kernel
+    zf, _ = aol.downscale_frame(x.unsqueeze(1))
+    assert torch.equal(zf[:, 0], z)
 
 
 @pytest.mark.parametrize("seed", range(30))
@@ -334,6 +337,11 @@ def test_bench_config_300_hd_frames(orc):
         zo, cso = run_oracle(orc, xh)
         assert np.array_equal(z[n:n + 1].cpu().numpy(), zo), n
         assert np_u64(cs[n:n + 1])[0] == cso[0]
+    # checksums of a spread of further frames (every 25th) against the oracle
+    got = np_u64(cs)
+    for n in range(12, 300, 25):
+        _, cso = run_oracle(orc, synth.frames(0, n, 1, C, H, W, "uniform"))
+        assert got[n] == cso[0], n
 
 
 def test_4k_batch(orc):
