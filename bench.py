@@ -208,7 +208,7 @@ def run_reference(a, rank):
     line = {
         "metric": METRIC, "value": value, "unit": "frames/s", "n_gpus": a.gpus, "steps": steps, "warmup": warm,
         "ms_per_step": 1000.0 * info["seconds"], "higher_is_better": True, "scaling": "weak",
-        "vs_baseline": None, "dtype": a.dtype, "data": "synthetic",
+        "vs_baseline": None, "dtype": "i32", "data": "synthetic",
         "config": {"workload": workload_name(a), "frames": a.frames, "H": a.H, "W": a.W,
                    "channels": a.channels, "l2": "inputs larger than L2 (no flush)"},
         "impl": "reference",
@@ -352,7 +352,7 @@ def main():
         "metric": METRIC, "value": value, "unit": "frames/s", "n_gpus": world, "steps": a.steps,
         "warmup": a.warmup, "ms_per_step": max_ms / a.steps, "higher_is_better": True,
         "scaling": "strong" if a.stream_frames else "weak",
-        "vs_baseline": None, "dtype": a.dtype, "data": "synthetic",
+        "vs_baseline": None, "dtype": "i32", "data": "synthetic",   # arithmetic type (uint8 samples are summed in int32)
         "config": {"workload": workload_name(a), "frames_per_gpu": count, "launches_per_step": len(calls),
                    "H": H, "W": W, "channels": C,
                    "in_dtype": a.dtype, "out_dtype": "i32", "l2": "inputs (7.46 GB at HD int32) larger than L2; no flush",

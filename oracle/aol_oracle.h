@@ -24,7 +24,9 @@
  * hand-derived ramp closed form, the constant-frame invariant, toroidal
  * shift-equivariance, locality, read-count histograms, pattern counts, output
  * shapes, C99 truncating-division tables.  The vertical filter (Z1/Z2) is a
- * reading: its tiler is pinned only by shapes, counts and invariants.
+ * reading: its tiler is pinned only by shapes, counts and invariants -- the
+ * oracle is pinned to the READING, but parity with the paper's own vertical
+ * taps is unpinned (the paper never prints them).
  */
 #ifndef AOL_ORACLE_H
 #define AOL_ORACLE_H
