@@ -227,6 +227,7 @@ aol_status_t make_tiler_dev(const aol_tiler_t* t, TilerDev* td) {
             order[last] = last;
         }
     }
+    td->small32 = td->linear && td->fast32 && td->array_elems < (int64_t(1) << 31) ? 1 : 0;
     int64_t gst[2 * AOL_MAX_RANK];
     int64_t g = 1;
     for (int d = td->nd - 1; d >= 0; --d) {

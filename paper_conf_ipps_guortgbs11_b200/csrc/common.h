@@ -76,6 +76,7 @@ struct TilerDev {
     int32_t ra, nd;             // array rank, combined (rep ++ pattern) rank
     int32_t linear;             // 1: no coordinate can wrap -> offset is affine in the tile index
     int32_t fast32;             // 1: total < 2^31 -> 32-bit magic-number division
+    int32_t small32;            // 1: linear, total and array offsets < 2^31 -> all-32-bit linear kernel
     uint32_t nowrap_mask;       // bit a: array dim a never wraps
     int64_t ext[2 * AOL_MAX_RANK];
     int64_t coef[AOL_MAX_RANK][2 * AOL_MAX_RANK];

@@ -190,6 +190,65 @@ __global__ void __launch_bounds__(256) tiler_kernel(const TilerDev td, const voi
     }
 }
 
+// Linear tilers whose array and tile offsets fit in 31 bits (the common case): the permuted walk with
+// all-32-bit digit arithmetic and the per-dimension constants staged once per CTA in shared memory
+// (one LDS.128 + one LDS per digit instead of five dynamically indexed constant-bank loads).
+template <int ES, int V, int MODE>
+__global__ void __launch_bounds__(256) tiler_linear32_kernel(const TilerDev td, const void* __restrict__ src,
+                                                             void* __restrict__ dst) {
+    using T = typename Elem<ES>::T;
+    using VT = typename Vec<ES * V>::T;
+    __shared__ int4 pk[kND];      // {extent, magic multiplier, shift, array stride}
+    __shared__ int32_t pg[kND];   // tile stride
+    if (threadIdx.x < td.nd) {
+        const int d = threadIdx.x;
+        pk[d] = make_int4(int32_t(td.p_ext[d]), int32_t(td.p_fd_mul[d]), int32_t(td.p_fd_shift[d]),
+                          int32_t(td.p_lin[d]));
+        pg[d] = int32_t(td.p_gst[d]);
+    }
+    __syncthreads();
+    const int32_t nvec = int32_t(td.total / V);
+    const int32_t stride = int32_t(gridDim.x * blockDim.x);
+    constexpr int kU = 4;
+    const int32_t warp_first = int32_t((blockIdx.x * blockDim.x + (threadIdx.x & ~31u)) * kU + (threadIdx.x & 31u));
+    for (int32_t v0 = warp_first; v0 < nvec; v0 += kU * stride) {
+        int32_t off[kU], g[kU];
+#pragma unroll
+        for (int u = 0; u < kU; ++u) {
+            const int32_t v = v0 + 32 * u;
+            uint32_t n = v < nvec ? uint32_t(v) * V : 0u;
+            int32_t o = int32_t(td.base), gg = 0;
+#pragma unroll 1
+            for (int d = td.nd - 1; d >= 0; --d) {
+                const int4 p = pk[d];
+                const uint32_t q = (__umulhi(n, uint32_t(p.y)) + n) >> p.z;
+                const int32_t i = int32_t(n - q * uint32_t(p.x));
+                n = q;
+                o += p.w * i;
+                gg += pg[d] * i;
+            }
+            off[u] = o;
+            g[u] = gg;
+        }
+        VT val[kU];
+        if (MODE == 0) {
+#pragma unroll
+            for (int u = 0; u < kU; ++u)
+                if (v0 + 32 * u < nvec) val[u] = reinterpret_cast<const VT*>(static_cast<const T*>(src) + off[u])[0];
+#pragma unroll
+            for (int u = 0; u < kU; ++u)
+                if (v0 + 32 * u < nvec) reinterpret_cast<VT*>(static_cast<T*>(dst) + g[u])[0] = val[u];
+        } else {
+#pragma unroll
+            for (int u = 0; u < kU; ++u)
+                if (v0 + 32 * u < nvec) val[u] = reinterpret_cast<const VT*>(static_cast<const T*>(src) + g[u])[0];
+#pragma unroll
+            for (int u = 0; u < kU; ++u)
+                if (v0 + 32 * u < nvec) reinterpret_cast<VT*>(static_cast<T*>(dst) + off[u])[0] = val[u];
+        }
+    }
+}
+
 int grid_for(int64_t n, int num_sms) {
     return int(std::max<int64_t>(1, std::min<int64_t>((n + 255) / 256, int64_t(num_sms) * 32)));
 }
@@ -198,6 +257,11 @@ template <int ES, int V, int MODE>
 aol_status_t launch_v(const TilerDev& td, const void* src, void* dst, unsigned long long* ws, int grid,
                       cudaStream_t s) {
     const bool fast = td.fast32 != 0, lin = td.linear != 0;
+    if (MODE <= 1 && lin && td.small32) {
+        tiler_linear32_kernel<ES, V, MODE><<<grid, 256, 0, s>>>(td, src, dst);
+        AOL_LAUNCH_CHECK("tiler_linear32_kernel");
+        return AOL_OK;
+    }
     if (fast && lin)
         tiler_kernel<ES, V, true, true, MODE><<<grid, 256, 0, s>>>(td, src, dst, ws);
     else if (fast)
