@@ -136,6 +136,93 @@ __global__ void __launch_bounds__(256) filter_kernel(const FilterDev fd, const i
     }
 }
 
+// All-32-bit variant for arrays < 2^31 elements whose reference-point sums fit in 31 bits (the usual
+// case): the pattern/output offset tables, read with a data-dependent index, are staged in shared
+// memory once per CTA instead of being fetched from the constant bank per element.
+template <int D>
+__global__ void __launch_bounds__(256) filter32_kernel(const FilterDev fd, const int32_t* __restrict__ in,
+                                                       int32_t* __restrict__ out) {
+    __shared__ int32_t lin_in[AOL_MAX_FILTER_PATTERN], lin_out[AOL_MAX_WINDOWS], start[AOL_MAX_WINDOWS];
+    if (threadIdx.x < AOL_MAX_FILTER_PATTERN) lin_in[threadIdx.x] = int32_t(fd.lin_in[threadIdx.x]);
+    if (threadIdx.x < AOL_MAX_WINDOWS) {
+        lin_out[threadIdx.x] = int32_t(fd.lin_out[threadIdx.x]);
+        start[threadIdx.x] = fd.start[threadIdx.x];
+    }
+    __syncthreads();
+    const int32_t nrep = int32_t(fd.nrep);
+    for (int32_t r = int32_t(blockIdx.x * blockDim.x + threadIdx.x); r < nrep; r += int32_t(gridDim.x * blockDim.x)) {
+        int32_t vi[D], vo[D];
+#pragma unroll
+        for (int a = 0; a < D; ++a) {
+            vi[a] = fd.o_in[a];
+            vo[a] = fd.o_out[a];
+        }
+        uint32_t n = uint32_t(r);
+#pragma unroll
+        for (int j = D - 1; j >= 0; --j) {
+            if (j < fd.rr) {
+                const uint32_t q = (__umulhi(n, fd.fd_mul[j]) + n) >> fd.fd_shift[j];
+                const int32_t i = int32_t(n - q * uint32_t(fd.rep_ext[j]));
+                n = q;
+#pragma unroll
+                for (int a = 0; a < D; ++a) {   // reference points o' + P'.r (Section IV)
+                    vi[a] += fd.P_in[a][j] * i;
+                    vo[a] += fd.P_out[a][j] * i;
+                }
+            }
+        }
+        bool in_ok = true, out_ok = true;
+        int32_t base_in = 0, base_out = 0;
+#pragma unroll
+        for (int a = 0; a < D; ++a) {
+            if (a < fd.ra_in) {
+                vi[a] %= fd.s_in[a];
+                in_ok &= vi[a] + fd.fmax_in[a] < fd.s_in[a];
+                base_in += vi[a] * int32_t(fd.st_in[a]);
+            }
+            if (a < fd.ra_out) {
+                vo[a] %= fd.s_out[a];
+                out_ok &= vo[a] + fd.fmax_out[a] < fd.s_out[a];
+                base_out += vo[a] * int32_t(fd.st_out[a]);
+            }
+        }
+        for (int k = 0; k < fd.n_win; ++k) {
+            int32_t S = 0;                                      // task (Fig. 5): tile = S/d - S%d
+            const int p0 = start[k];
+            if (in_ok) {
+                for (int t = 0; t < fd.len; ++t) S += __ldg(in + base_in + lin_in[p0 + t]);
+            } else {
+                for (int t = 0; t < fd.len; ++t) {
+                    int32_t off = 0;
+#pragma unroll
+                    for (int a = 0; a < D; ++a) {
+                        if (a < fd.ra_in) {
+                            int32_t c = vi[a] + fd.f_in[p0 + t][a];   // toroidal pattern element
+                            if (c >= fd.s_in[a]) c -= fd.s_in[a];
+                            off += c * int32_t(fd.st_in[a]);
+                        }
+                    }
+                    S += __ldg(in + off);
+                }
+            }
+            const int32_t tile = S / fd.divisor - S % fd.divisor;
+            int32_t off = base_out + lin_out[k];
+            if (!out_ok) {
+                off = 0;
+#pragma unroll
+                for (int a = 0; a < D; ++a) {
+                    if (a < fd.ra_out) {
+                        int32_t c = vo[a] + fd.f_out[k][a];
+                        if (c >= fd.s_out[a]) c -= fd.s_out[a];
+                        off += c * int32_t(fd.st_out[a]);
+                    }
+                }
+            }
+            out[off] = tile;
+        }
+    }
+}
+
 int64_t emod(int64_t a, int64_t m) {
     const int64_t r = a % m;
     return r < 0 ? r + m : r;
@@ -314,6 +401,23 @@ aol_status_t aol_filter_apply(const aol_filter_t* f, const int32_t* d_in, int32_
     if (st != AOL_OK) return st;
     const int grid = int(std::max<int64_t>(1, std::min<int64_t>((fd.nrep + 255) / 256, int64_t(dev.num_sms) * 16)));
     const int D = std::max(fd.rr, std::max(fd.ra_in, fd.ra_out));
+    // all-32-bit path: arrays < 2^31 elements, repetitions < 2^31, reference-point sums < 2^31
+    bool small = fd.fast32 && elems(f->in.array_shape, f->in.array_rank) < (int64_t(1) << 31) &&
+                 elems(f->out.array_shape, f->out.array_rank) < (int64_t(1) << 31);
+    for (const aol_tiler_t* t : {&f->in, &f->out})
+        for (int a = 0; a < t->array_rank; ++a) {
+            __int128 bound = t->array_shape[a];
+            for (int j = 0; j < t->rep_rank; ++j) bound += __int128(t->array_shape[a]) * t->rep_shape[j];
+            if (bound >= (__int128(1) << 31)) small = false;
+        }
+    if (small) {
+        if (D <= 2) filter32_kernel<2><<<grid, 256, 0, s>>>(fd, d_in, d_out);
+        else if (D <= 3) filter32_kernel<3><<<grid, 256, 0, s>>>(fd, d_in, d_out);
+        else if (D <= 4) filter32_kernel<4><<<grid, 256, 0, s>>>(fd, d_in, d_out);
+        else filter32_kernel<8><<<grid, 256, 0, s>>>(fd, d_in, d_out);
+        AOL_LAUNCH_CHECK("filter32_kernel");
+        return AOL_OK;
+    }
     auto launch = [&](auto kfast, auto kd) {
         filter_kernel<decltype(kd)::value, decltype(kfast)::value><<<grid, 256, 0, s>>>(fd, d_in, d_out);
     };
