@@ -178,7 +178,8 @@ AOL_API aol_status_t aol_tiler_scatter(const aol_tiler_t* t, aol_dtype_t el, con
 
 /* Horizontal filter alone (the SaC/GASPARD2 "HorizontalFilter", Fig. 10 tilers
  * + Fig. 5 task): d_in int32 [planes][H][W] -> d_out int32 [planes][H][3W/8].
- * W % 8 == 0 else AOL_E_SHAPE.  Pointers 16-byte aligned.  Async on s. */
+ * W % 8 == 0 else AOL_E_SHAPE.  Pointers 4-byte aligned (a 16-byte aligned input takes the
+ * 128-bit vector path).  Async on s. */
 AOL_API aol_status_t aol_downscale_h(const int32_t* d_in, int32_t* d_out, int64_t planes, int64_t H, int64_t W,
                              cudaStream_t s);
 

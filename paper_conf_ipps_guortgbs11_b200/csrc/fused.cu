@@ -212,7 +212,10 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
     a.Z = d_out;
     a.cs = d_cs;
     a.X = d_in;
-    a.nunits = plan.units;
+    // units from THIS call's frame count (a plan may be reused for a shorter batch, e.g. the last chunk of
+    // the host-streamed path): never more units, or CTAs, than the batch has
+    a.nunits = planes * plan.units_per_plane;
+    const int grid = int(std::min<int64_t>(plan.grid, a.nunits));
     a.H = int32_t(H);
     a.W = int32_t(W);
     a.Ho = Ho;
@@ -239,7 +242,7 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
     KernelFn k = pick(in_dtype, d_cs != nullptr, plan.block, plan.ctas_per_sm);
     aol_status_t st_attr = kernel_smem(reinterpret_cast<const void*>(k), plan.smem);
     if (st_attr != AOL_OK) return st_attr;
-    k<<<plan.grid, plan.block, plan.smem, s>>>(map, a);
+    k<<<grid, plan.block, plan.smem, s>>>(map, a);
     AOL_LAUNCH_CHECK("fused_tma_kernel");
     return AOL_OK;
 }

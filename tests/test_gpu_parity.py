@@ -366,6 +366,23 @@ def test_host_streamed_matches_device(orc):
     assert np.array_equal(csh.view(torch.int64).numpy().view(np.uint64), cso)
 
 
+@pytest.mark.parametrize("chunk", [1, 4, 7, 50])
+def test_host_streamed_u8_and_ragged_chunks(orc, chunk):
+    """uint8 samples from pageable and pinned host memory; chunk sizes that do not divide the batch."""
+    N, C, H, W = 7, 3, 36, 256
+    xh = synth.frames(13, 0, N, C, H, W)
+    zo, cso = run_oracle(orc, xh)
+    for pinned in (False, True):
+        x8 = torch.from_numpy(xh.astype(np.uint8))
+        if pinned:
+            x8 = x8.pin_memory()
+        zh, csh = aol.downscale_frame_host(x8, chunk_frames=chunk)
+        assert np.array_equal(zh.numpy(), zo)
+        assert np.array_equal(csh.view(torch.int64).numpy().view(np.uint64), cso)
+    zh, csh = aol.downscale_frame_host(torch.from_numpy(xh), chunk_frames=chunk, checksums=False)
+    assert csh is None and np.array_equal(zh.numpy(), zo)
+
+
 # -------------------------------------------------------------- edge cases
 
 @pytest.mark.parametrize("W,dtype,kernel", [(7680, torch.int32, 1), (7936, torch.int32, 2), (7936, torch.uint8, 1),
