@@ -52,6 +52,50 @@ KernelFn pick(aol_dtype_t dt, bool checksum, int block, int cps) {
     return dt == AOL_U8 ? tma_kernel_u8(checksum, block, cps) : tma_kernel_i32(checksum, block, cps);
 }
 
+// Shared-memory geometry of the TMA ring: one stage = one row triple.
+struct RingGeom {
+    uint32_t stage_bytes;   // 3 rows of the input
+    uint32_t stage_stride;  // rounded up: 1024 B (SWIZZLE_128B atom) for int32, 128 B for uint8
+    uint32_t out_bytes;     // one band of output: 4 rows of Wo int32
+};
+
+RingGeom ring_geom(aol_dtype_t dt, int64_t W) {
+    const uint32_t es = dt == AOL_U8 ? 1u : 4u, align = dt == AOL_U8 ? 128u : 1024u;
+    RingGeom g;
+    g.stage_bytes = uint32_t(3 * W) * es;
+    g.stage_stride = (g.stage_bytes + align - 1) & ~(align - 1);
+    g.out_bytes = uint32_t(16 * (3 * (W / 8)));
+    return g;
+}
+
+// ring + output staging + full/empty mbarriers + checksum partials + 1 KB alignment slack
+int smem_bytes(const RingGeom& g, int stages) {
+    return stages * int(g.stage_stride) + kOutBufs * int(g.out_bytes) + 2 * stages * 8 + 256 + 1024;
+}
+
+// TMA descriptor for row triples of a [rows][W] array viewed as {inner, W/inner, rows}: int32 with a
+// 128 B swizzle (inner = 32 elements), uint8 unswizzled (inner = 128 elements).
+aol_status_t encode_row_map(CUtensorMap* map, aol_dtype_t dt, const void* base, int64_t rows, int64_t W) {
+    EncodeTiledFn encode;
+    aol_status_t st = get_encode_fn(&encode);
+    if (st != AOL_OK) return st;
+    const bool i32 = dt == AOL_I32;
+    const cuuint64_t inner = i32 ? 32 : 128, es = i32 ? 4 : 1;
+    const cuuint64_t gdim[3] = {inner, cuuint64_t(W) / inner, cuuint64_t(rows)};
+    const cuuint64_t gstride[2] = {inner * es, cuuint64_t(W) * es};
+    const cuuint32_t box[3] = {cuuint32_t(inner), cuuint32_t(W / int64_t(inner)), 3};
+    const cuuint32_t estr[3] = {1, 1, 1};
+    CUresult cr = encode(map, i32 ? CU_TENSOR_MAP_DATA_TYPE_INT32 : CU_TENSOR_MAP_DATA_TYPE_UINT8, 3,
+                         const_cast<void*>(base), gdim, gstride, box, estr, CU_TENSOR_MAP_INTERLEAVE_NONE,
+                         i32 ? CU_TENSOR_MAP_SWIZZLE_128B : CU_TENSOR_MAP_SWIZZLE_NONE,
+                         CU_TENSOR_MAP_L2_PROMOTION_L2_256B, CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+    if (cr != CUDA_SUCCESS) {
+        set_error("cuTensorMapEncodeTiled failed (CUresult %d)", int(cr));
+        return AOL_E_CUDA;
+    }
+    return AOL_OK;
+}
+
 }  // namespace
 
 aol_status_t plan_fused(aol_dtype_t in_dtype, const void* d_in, const int32_t* d_out, int64_t frames,
@@ -67,11 +111,7 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, const void* d_in, const int32_t* d
 
     bool tma_ok = tma_shape_ok(in_dtype, planes, channels, H, W) && (d_in == nullptr || aligned16(d_in)) &&
                   (d_out == nullptr || aligned16(d_out));
-    const int es = in_dtype == AOL_U8 ? 1 : 4;
-    const uint32_t stage_bytes = uint32_t(3 * W * es);
-    const uint32_t align = in_dtype == AOL_U8 ? 128u : 1024u;
-    const uint32_t stage_stride = (stage_bytes + align - 1) & ~(align - 1);
-    const uint32_t out_bytes = uint32_t(16 * Wo);
+    const RingGeom geom = ring_geom(in_dtype, W);
     const int nc = int(((W / 8) + 31) / 32 * 32);
     const int block = nc + 32;
     int stages = 0, cps = 1;
@@ -86,17 +126,18 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, const void* d_in, const int32_t* d
                                 : std::max(1, std::min(8, (want_warps + cwarps - 1) / cwarps));
         for (;; --cps) {
             const int budget = std::min(dev.smem_optin, dev.smem_per_sm / cps - 1024);
-            const int fixed = kOutBufs * int(out_bytes) + 2 * kMaxStages * 8 + 256 + 1024;  // out, barriers, red, slack
-            stages = std::min((budget - fixed) / int(stage_stride), kMaxStages);
+            const int fixed = smem_bytes(geom, 0) + 2 * kMaxStages * 8;   // everything but the ring itself
+            stages = std::min((budget - fixed) / int(geom.stage_stride), kMaxStages);
             if (o.stages > 0) {
                 stages = std::min(stages, o.stages);
             } else {
-                const int target = (kInflightBytesPerSM / cps + int(stage_stride) / 2) / int(stage_stride);
+                const int target = (kInflightBytesPerSM / cps + int(geom.stage_stride) / 2) / int(geom.stage_stride);
                 stages = std::min(stages, std::max(2, target));
             }
             int occ = 0;
-            const int smem = stages * int(stage_stride) + kOutBufs * int(out_bytes) + 2 * stages * 8 + 256 + 1024;
-            if (stages >= 2 && cps > 1) occ = kernel_occupancy(reinterpret_cast<const void*>(pick(in_dtype, true, block, cps)), block, smem);
+            const int smem = smem_bytes(geom, stages);
+            if (stages >= 2 && cps > 1)
+                occ = kernel_occupancy(reinterpret_cast<const void*>(pick(in_dtype, true, block, cps)), block, smem);
             if (cps == 1) occ = 1;   // one CTA always fits once its shared memory does
             if ((stages >= 2 && occ >= cps) || cps == 1 || o.ctas_per_sm > 0) {
                 if (stages < 2) tma_ok = false;
@@ -137,7 +178,7 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, const void* d_in, const int32_t* d
         plan->grid = int(std::min<int64_t>(plan->units, max_ctas));
         plan->block = block;
         plan->stages = stages;
-        plan->smem = stages * int(stage_stride) + kOutBufs * int(out_bytes) + 2 * stages * 8 + 256 + 1024;
+        plan->smem = smem_bytes(geom, stages);
         plan->ctas_per_sm = cps;
         plan->flags = o.flags;
     } else {
@@ -173,39 +214,11 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
 
     CUtensorMap map;
     std::memset(&map, 0, sizeof map);
-    if (in_dtype == AOL_I32) {
-        EncodeTiledFn encode;
-        aol_status_t st = get_encode_fn(&encode);
-        if (st != AOL_OK) return st;
-        const cuuint64_t gdim[3] = {32, cuuint64_t(W / 32), cuuint64_t(planes * H)};
-        const cuuint64_t gstride[2] = {128, cuuint64_t(W) * 4};
-        const cuuint32_t box[3] = {32, cuuint32_t(W / 32), 3};
-        const cuuint32_t estr[3] = {1, 1, 1};
-        CUresult cr = encode(&map, CU_TENSOR_MAP_DATA_TYPE_INT32, 3, const_cast<void*>(d_in), gdim, gstride, box,
-                             estr, CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_128B,
-                             CU_TENSOR_MAP_L2_PROMOTION_L2_256B, CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
-        if (cr != CUDA_SUCCESS) {
-            set_error("cuTensorMapEncodeTiled failed (CUresult %d)", int(cr));
-            return AOL_E_CUDA;
-        }
-    }
     const bool u8_tensor = in_dtype == AOL_U8 && W % 128 == 0 && W / 128 <= 256 &&
                            planes * H < (int64_t(1) << 31) && !(plan.flags & AOL_FLAG_U8_BULK);
-    if (u8_tensor) {
-        EncodeTiledFn encode;
-        aol_status_t st = get_encode_fn(&encode);
+    if (in_dtype == AOL_I32 || u8_tensor) {
+        aol_status_t st = encode_row_map(&map, in_dtype, d_in, planes * H, W);
         if (st != AOL_OK) return st;
-        const cuuint64_t gdim[3] = {128, cuuint64_t(W / 128), cuuint64_t(planes * H)};
-        const cuuint64_t gstride[2] = {128, cuuint64_t(W)};
-        const cuuint32_t box[3] = {128, cuuint32_t(W / 128), 3};
-        const cuuint32_t estr[3] = {1, 1, 1};
-        CUresult cr = encode(&map, CU_TENSOR_MAP_DATA_TYPE_UINT8, 3, const_cast<void*>(d_in), gdim, gstride, box,
-                             estr, CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE,
-                             CU_TENSOR_MAP_L2_PROMOTION_L2_256B, CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
-        if (cr != CUDA_SUCCESS) {
-            set_error("cuTensorMapEncodeTiled (uint8) failed (CUresult %d)", int(cr));
-            return AOL_E_CUDA;
-        }
     }
     FusedArgs a;
     a.u8_tensor = u8_tensor ? 1 : 0;
@@ -228,11 +241,10 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
     a.bands_per_unit = plan.bands_per_unit;
     a.units_per_plane = plan.units_per_plane;
     a.stages = plan.stages;
-    const int es = in_dtype == AOL_U8 ? 1 : 4;
-    const uint32_t align = in_dtype == AOL_U8 ? 128u : 1024u;
-    a.stage_bytes = uint32_t(3 * W * es);
-    a.stage_stride = (a.stage_bytes + align - 1) & ~(align - 1);
-    a.out_bytes = uint32_t(16 * Wo);
+    const RingGeom geom = ring_geom(in_dtype, W);
+    a.stage_bytes = geom.stage_bytes;
+    a.stage_stride = geom.stage_stride;
+    a.out_bytes = geom.out_bytes;
     a.n_consumer = plan.block - 32;
     a.halo_last = (plan.flags & AOL_FLAG_HALO_LAST) ? 1 : 0;
     a.hint_loads = (plan.flags & AOL_FLAG_EVICT_FIRST_LOADS) ? 1 : 0;
