@@ -101,6 +101,51 @@ __global__ void __launch_bounds__(256) downscale_v_kernel(const int32_t* __restr
     }
 }
 
+// Vectorised K-4 (W % 4 == 0, 16-byte aligned): thread per (plane, run of kVBands bands, 4 adjacent
+// columns).  It walks its bands top to bottom with 128-bit loads, carrying rows 9..11 of band b over as
+// rows 0..2 of band b+1, so every Y row is loaded once per thread (plus the 3 halo rows of the run).
+constexpr int kVBands = 8;
+
+__global__ void __launch_bounds__(256) downscale_v_vec_kernel(const int32_t* __restrict__ Y, int32_t* __restrict__ Z,
+                                                              int64_t planes, int32_t H, int32_t W) {
+    const int32_t nb = H / 9, Q = W / 4, nchunks = (nb + kVBands - 1) / kVBands;
+    const int64_t total = planes * nchunks * Q;
+    for (int64_t i = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; i < total; i += int64_t(gridDim.x) * blockDim.x) {
+        const int32_t q = int32_t(i % Q);
+        const int64_t rest = i / Q;
+        const int32_t c = int32_t(rest % nchunks);
+        const int64_t plane = rest / nchunks;
+        const int4* yp = reinterpret_cast<const int4*>(Y + size_t(plane) * H * W) + q;
+        int4* zp = reinterpret_cast<int4*>(Z + size_t(plane) * (4 * nb) * W) + q;
+        const int32_t b0 = c * kVBands, b1 = min(b0 + kVBands, nb);
+        int4 v[12];
+#pragma unroll
+        for (int j = 0; j < 3; ++j) v[j] = __ldg(yp + size_t(9 * b0 + j) * Q);
+        for (int32_t b = b0; b < b1; ++b) {
+#pragma unroll
+            for (int j = 3; j < 12; ++j) {
+                int32_t row = 9 * b + j;
+                if (row >= H) row -= H;   // the last band's halo wraps to rows 0..2 (reading Z1)
+                v[j] = __ldg(yp + size_t(row) * Q);
+            }
+#pragma unroll
+            for (int k = 0; k < 4; ++k) {
+                int4 S = v[2 * k];
+#pragma unroll
+                for (int t = 1; t < 6; ++t) {
+                    S.x += v[2 * k + t].x;
+                    S.y += v[2 * k + t].y;
+                    S.z += v[2 * k + t].z;
+                    S.w += v[2 * k + t].w;
+                }
+                zp[size_t(4 * b + k) * Q] = make_int4(task_T(S.x), task_T(S.y), task_T(S.z), task_T(S.w));
+            }
+#pragma unroll
+            for (int j = 0; j < 3; ++j) v[j] = v[9 + j];
+        }
+    }
+}
+
 // cs[f] += sum_e (u64)(u32)Z[f][e] * (e + 1)   (e = flat index within the frame)
 __global__ void __launch_bounds__(256) checksum_kernel(const int32_t* __restrict__ Z, int64_t frames,
                                                        int64_t per_frame, uint64_t* __restrict__ cs) {
@@ -145,6 +190,13 @@ aol_status_t launch_downscale_v(const int32_t* d_in, int32_t* d_out, int64_t pla
     DeviceInfo dev;
     aol_status_t st = device_info(&dev);
     if (st != AOL_OK) return st;
+    if (W % 4 == 0 && aligned16(d_in) && aligned16(d_out)) {
+        const int64_t total = planes * ((H / 9 + kVBands - 1) / kVBands) * (W / 4);
+        const int grid = int(std::max<int64_t>(1, std::min<int64_t>((total + 255) / 256, int64_t(dev.num_sms) * 16)));
+        downscale_v_vec_kernel<<<grid, 256, 0, s>>>(d_in, d_out, planes, int32_t(H), int32_t(W));
+        AOL_LAUNCH_CHECK("downscale_v_vec_kernel");
+        return AOL_OK;
+    }
     const int64_t total = planes * (H / 9) * W;
     const int grid = int(std::max<int64_t>(1, std::min<int64_t>((total + 255) / 256, int64_t(dev.num_sms) * 16)));
     downscale_v_kernel<<<grid, 256, 0, s>>>(d_in, d_out, planes, int32_t(H), int32_t(W));
