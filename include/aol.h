@@ -107,7 +107,7 @@ typedef struct {
     int32_t flags;          /* AOL_FLAG_* bits (tuning experiments; results are identical)    */
 } aol_launch_opts_t;
 
-#define AOL_FLAG_HALO_LAST 1           /* stream a unit's 3 halo rows after its own rows, not first */
+/* bit 0 is reserved (was AOL_FLAG_HALO_LAST, a round-1 experiment: the halo rows now always stream first) */
 #define AOL_FLAG_EVICT_FIRST_LOADS 2   /* TMA input loads with the L2 evict_first policy            */
 #define AOL_FLAG_EVICT_FIRST_STORES 4  /* TMA output stores with the L2 evict_first policy          */
 #define AOL_FLAG_BLOCKED_UNITS 8       /* each CTA takes a contiguous block of work units (default:

@@ -246,7 +246,6 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
     a.stage_stride = geom.stage_stride;
     a.out_bytes = geom.out_bytes;
     a.n_consumer = plan.block - 32;
-    a.halo_last = (plan.flags & AOL_FLAG_HALO_LAST) ? 1 : 0;
     a.hint_loads = (plan.flags & AOL_FLAG_EVICT_FIRST_LOADS) ? 1 : 0;
     a.hint_stores = (plan.flags & AOL_FLAG_EVICT_FIRST_STORES) ? 1 : 0;
     a.blocked_units = (plan.flags & AOL_FLAG_BLOCKED_UNITS) ? 1 : 0;

@@ -53,10 +53,10 @@ constexpr int kMaxConsumers = 992;  // + 1 producer warp = 1024 threads
 // band has long finished reading smem by the time the next band (3 triples
 // later) is emitted, and the saved space buys one more ring stage.
 constexpr int kOutBufs = 1;
-// Bytes of TMA loads to keep in flight per SM.  Measured on B200
-// (profiles/r01_stage_sweep.jsonl): HD int32 throughput peaks at 6 row-triples
-// (138 KB) per SM; deeper rings are SLOWER (9 stages: -5%), shallower starve HBM.
-constexpr int kInflightBytesPerSM = 6 * 23552;
+// Bytes of TMA loads to keep in flight per SM.  Measured on B200 (profiles/r01_stage_sweep*.jsonl): HD
+// int32 throughput peaks at 5 row-triples (115 KB) per SM with the band-unrolled consumer (it was 6 with
+// the slower first consumer); deeper rings are SLOWER (HBM efficiency drops), shallower starve HBM.
+constexpr int kInflightBytesPerSM = 5 * 23552;
 
 __device__ __forceinline__ int32_t task_T(int32_t S) {
     // Fig. 5: tmp/6 - tmp%6 == 7*(tmp/6) - tmp for C truncating division.
@@ -88,7 +88,6 @@ struct FusedArgs {
     uint32_t stage_stride;  // stage_bytes rounded up (1024 for the swizzle atom, 128 for uint8)
     uint32_t out_bytes;     // 16*Wo  (4 output rows)
     int32_t n_consumer;     // consumer threads, multiple of 32
-    int32_t halo_last;      // 1: stream the halo triple after the unit's own rows
     int32_t hint_loads;     // 1: TMA loads with L2 evict_first (input is streamed once)
     int32_t hint_stores;    // 1: bulk stores with L2 evict_first
     int32_t blocked_units;  // 1: contiguous block of units per CTA instead of round-robin
@@ -192,8 +191,7 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
                 // halo triple: rows 9*b1 .. 9*b1+2 (mod H -- the V tiler's toroidal wrap for the last band)
                 const int32_t halo = (3 * b1 == a.triples_per_plane) ? 0 : 3 * b1;
                 for (int32_t t = 0; t < ntrip; ++t) {
-                    const int32_t trip = a.halo_last ? (t == ntrip - 1 ? halo : 3 * b0 + t)
-                                                     : (t == 0 ? halo : 3 * b0 + t - 1);
+                    const int32_t trip = t == 0 ? halo : 3 * b0 + t - 1;
                     ptx::mbar_wait_sleep(&empty[s], ph ^ 1u);   // suspended, not spinning, while the ring is full
                     ptx::mbar_arrive_expect_tx(&full[s], a.stage_bytes);
                     uint8_t* dst = stage_base + size_t(s) * a.stage_stride;
@@ -252,7 +250,6 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
         const int64_t plane = u / a.units_per_plane;
         const int32_t b0 = int32_t(u - plane * a.units_per_plane) * a.bands_per_unit;
         const int32_t b1 = min(b0 + a.bands_per_unit, a.nbands);
-        const int32_t ntrip = 3 * (b1 - b0) + 1;
         const int32_t chan = int32_t(plane % a.channels);
         uint64_t csacc = 0;
 
@@ -305,15 +302,10 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
             }
         };
 
-        int tau = 0;
-        for (int32_t ti = 0; ti < ntrip; ++ti) {
-            // logical triple index: 0 = halo, 1.. = the unit's own triples in order
-            const int32_t t = a.halo_last ? (ti == ntrip - 1 ? 0 : ti + 1) : ti;
+        // Wait for the next ring stage, run the H stage on its 3 rows (y[row][col]), release the stage.
+        auto triple = [&](int32_t (&y)[3][3]) {
             ptx::mbar_wait_sleep(&full[s], ph);
             const uint32_t sb = stage_s32 + uint32_t(s) * a.stage_stride;   // 32-bit shared address
-
-            // ---- H stage on the 3 rows of this triple: y[row][col]
-            int32_t y[3][3];
 #pragma unroll
             for (int rr = 0; rr < 3; ++rr) {
 #ifdef AOL_PROBE_STREAM_ONLY
@@ -330,51 +322,52 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
                 s = 0;
                 ph ^= 1u;
             }
+        };
 
-            if (t == 0) {   // the halo triple: keep what the last band needs from it
+        {   // the halo triple comes first: keep what the unit's last band needs from it (rows 9 and 9..11)
+            int32_t y[3][3];
+            triple(y);
 #pragma unroll
-                for (int m = 0; m < 3; ++m) {
-                    Hr9[m] = y[0][m];
-                    Hr911[m] = y[0][m] + y[1][m] + y[2][m];
-                }
-                continue;
+            for (int m = 0; m < 3; ++m) {
+                Hr9[m] = y[0][m];
+                Hr911[m] = y[0][m] + y[1][m] + y[2][m];
             }
-
-            // ---- V stage: running sums of the 12-row pattern (windows start at rows 0,2,4,6)
-            if (tau == 0) {
-                if (t > 1) {
-                    // rows 0..2 of this band are rows 9..11 of the previous one: emit it
-                    int32_t r9[3], r911[3];
-#pragma unroll
-                    for (int m = 0; m < 3; ++m) {
-                        r9[m] = y[0][m];
-                        r911[m] = y[0][m] + y[1][m] + y[2][m];
-                    }
-                    emit(b0 + (t - 1) / 3 - 1, r9, r911);
-                }
+        }
+        // ---- one band per iteration; V stage = running sums of the 12-row pattern (windows at rows 0,2,4,6)
+        for (int32_t band = b0; band < b1; ++band) {
+            int32_t y[3][3];
+            triple(y);   // rows 0..2
+            if (band > b0) {
+                // rows 0..2 of this band are rows 9..11 of the previous one: emit it
+                int32_t r9[3], r911[3];
 #pragma unroll
                 for (int m = 0; m < 3; ++m) {
-                    A0[m] = y[0][m] + y[1][m] + y[2][m];   // rows 0..2 of window 0..5
-                    A1[m] = y[2][m];                        // row 2 of window 2..7
+                    r9[m] = y[0][m];
+                    r911[m] = y[0][m] + y[1][m] + y[2][m];
                 }
-            } else if (tau == 1) {
-#pragma unroll
-                for (int m = 0; m < 3; ++m) {
-                    const int32_t s3 = y[0][m] + y[1][m] + y[2][m];   // rows 3..5
-                    A0[m] += s3;
-                    A1[m] += s3;
-                    A2[m] = y[1][m] + y[2][m];                        // rows 4,5 of window 4..9
-                }
-            } else {
-#pragma unroll
-                for (int m = 0; m < 3; ++m) {
-                    const int32_t s2 = y[0][m] + y[1][m];             // rows 6,7
-                    A1[m] += s2;
-                    A2[m] += s2 + y[2][m];
-                    A3[m] = s2 + y[2][m];                             // rows 6..8 of window 6..11
-                }
+                emit(band - 1, r9, r911);
             }
-            if (++tau == 3) tau = 0;
+#pragma unroll
+            for (int m = 0; m < 3; ++m) {
+                A0[m] = y[0][m] + y[1][m] + y[2][m];   // rows 0..2 of window 0..5
+                A1[m] = y[2][m];                        // row 2 of window 2..7
+            }
+            triple(y);   // rows 3..5
+#pragma unroll
+            for (int m = 0; m < 3; ++m) {
+                const int32_t s3 = y[0][m] + y[1][m] + y[2][m];
+                A0[m] += s3;
+                A1[m] += s3;
+                A2[m] = y[1][m] + y[2][m];                        // rows 4,5 of window 4..9
+            }
+            triple(y);   // rows 6..8
+#pragma unroll
+            for (int m = 0; m < 3; ++m) {
+                const int32_t s2 = y[0][m] + y[1][m];
+                A1[m] += s2;
+                A2[m] += s2 + y[2][m];
+                A3[m] = s2 + y[2][m];                             // rows 6..8 of window 6..11
+            }
         }
         emit(b1 - 1, Hr9, Hr911);   // the unit's last band, completed by the halo rows
 

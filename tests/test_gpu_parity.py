@@ -79,7 +79,8 @@ def test_fused_vs_oracle(orc, shape, kernel):
 @pytest.mark.parametrize("opts", [
     {"bands_per_unit": 1}, {"bands_per_unit": 2}, {"bands_per_unit": 7}, {"bands_per_unit": 40},
     {"stages": 2}, {"stages": 3, "bands_per_unit": 5}, {"ctas_per_sm": 2}, {"ctas_per_sm": 2, "stages": 2},
-    {"flags": 1}, {"flags": 1, "bands_per_unit": 1, "stages": 2}, {"ctas_per_sm": 4}, {"ctas_per_sm": 8, "stages": 2},
+    {"flags": 8}, {"flags": 8, "bands_per_unit": 1, "stages": 2}, {"ctas_per_sm": 4}, {"ctas_per_sm": 8, "stages": 2},
+    {"flags": 2}, {"flags": 4},
 ])
 def test_fused_launch_options(orc, opts):
     """Unit boundaries, ring wrap-around and CTA residency do not change results."""
@@ -136,7 +137,8 @@ def test_fused_u8_launch_options(orc):
     xh = synth.frames(22, 0, 3, 3, 117, 512, "uniform")
     zo, cso = run_oracle(orc, xh)
     x8 = torch.from_numpy(xh.astype(np.uint8)).cuda()
-    for o in ({"bands_per_unit": 1}, {"stages": 2}, {"ctas_per_sm": 2}, {"ctas_per_sm": 4}, {"flags": 1}):
+    for o in ({"bands_per_unit": 1}, {"stages": 2}, {"ctas_per_sm": 2}, {"ctas_per_sm": 4}, {"flags": 16},
+              {"flags": 24, "bands_per_unit": 3}):
         z, cs = aol.downscale_frame(x8, checksums=True, opts=dict(o, kernel=1))
         torch.cuda.synchronize()
         assert np.array_equal(z.cpu().numpy(), zo), o
