@@ -249,10 +249,6 @@ aol_status_t make_tiler_dev(const aol_tiler_t* t, TilerDev* td) {
 
 using namespace aol;
 
-namespace aol {
-const char* last_error_cstr();
-}
-
 namespace {
 
 aol_status_t check_frame_args(const void* d_in, aol_dtype_t in_dtype, const int32_t* d_out, int64_t frames,

@@ -13,6 +13,7 @@ namespace aol {
 // Thread-local last-error message (besides the memos in api.cu, the library's only mutable state).
 void set_error(const char* fmt, ...) __attribute__((format(printf, 1, 2)));
 void clear_error();
+const char* last_error_cstr();
 
 inline aol_status_t fail(aol_status_t st, const char* what) {
     set_error("%s", what);
