@@ -183,7 +183,7 @@ def test_frame_checksum_kernel(orc):
 
 # -------------------------------------------------------------- generic tilers
 
-@pytest.mark.parametrize("seed", range(60))
+@pytest.mark.parametrize("seed", range(200))
 def test_tiler_gather_scatter_vs_oracle(orc, seed):
     rng = np.random.default_rng(5000 + seed)
     d = bf.random_descriptor(rng)
@@ -265,7 +265,7 @@ def test_filter_presets_vs_oracle(orc, shape):
     assert torch.equal(zf[:, 0], z)
 
 
-@pytest.mark.parametrize("seed", range(30))
+@pytest.mark.parametrize("seed", range(60))
 def test_filter_random_tilers_vs_oracle(orc, seed):
     """f3 with random input/output tilers and the paper's task windows: equal to the oracle's
     gather -> task_h/task_v -> scatter (Fig. 4, 5, 6) on the same descriptors."""
