@@ -21,6 +21,18 @@ def golden(name):
         return json.load(f)
 
 
+@pytest.fixture(scope="session", autouse=True)
+def ensure_built():
+    """Build libaol.so / liboracle.so / the C example if a checkout arrives without them (they are
+    git-ignored build products)."""
+    pkg = os.path.join(ROOT, "paper_conf_ipps_guortgbs11_b200", "libaol.so")
+    if not (os.path.exists(pkg) and os.path.exists(os.path.join(ROOT, "oracle", "liboracle.so"))):
+        import __graft_entry__
+
+        __graft_entry__.build()
+    yield
+
+
 @pytest.fixture(scope="session")
 def orc():
     import oracle
