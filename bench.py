@@ -56,6 +56,8 @@ def parse():
     p.add_argument("--e2e-steps", type=int, default=3)
     p.add_argument("--no-e2e", action="store_true")
     p.add_argument("--no-cpu-baseline", action="store_true")
+    p.add_argument("--dump-checksums", type=str, default="",
+                   help="rank 0 saves the gathered per-frame checksums (global frame order, .npy) for the tests")
     return p.parse_args()
 
 
@@ -303,6 +305,8 @@ def main():
               if a.stream_frames else None)
     max_ms, cs_all_t = shard.gather_results(cs if backend == "nccl" else cs.cpu(), elapsed_ms, counts=counts)
     cs_all = cs_all_t.cpu().numpy().view(np.uint64) if world > 1 else None
+    if a.dump_checksums and rank == 0:
+        np.save(a.dump_checksums, cs_all if cs_all is not None else cs.cpu().view(torch.int64).numpy().view(np.uint64))
 
     # e2e through the host-buffer C-ABI call
     e2e = None

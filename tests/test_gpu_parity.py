@@ -347,15 +347,25 @@ def test_bench_config_300_hd_frames(orc):
 
 
 def test_4k_batch(orc):
-    """BASELINE configs[3]: 3840x2160 frames, same ratios (sampled frames vs oracle)."""
-    N, C, H, W = 16, 3, 2160, 3840
+    """BASELINE configs[3]: the 64-frame 3840x2160 batch tools/bench_configs.py times.
+    Frames {0, 63} element by element against the oracle; every frame's fused checksum against the
+    stand-alone checksum kernel; a spread of checksums against the oracle."""
+    N, C, H, W = 64, 3, 2160, 3840
     x = aol.synth_frames(1, 0, N, C, H, W, "uniform")
     z, cs = aol.downscale_frame(x, checksums=True)
+    cs2 = aol.frame_checksum(z)
     torch.cuda.synchronize()
+    assert torch.equal(cs.view(torch.int64), cs2.view(torch.int64))
+    got = np_u64(cs)
     for n in (0, N - 1):
         zo, cso = run_oracle(orc, synth.frames(1, n, 1, C, H, W, "uniform"))
         assert np.array_equal(z[n:n + 1].cpu().numpy(), zo)
-        assert np_u64(cs[n:n + 1])[0] == cso[0]
+        assert got[n] == cso[0]
+    for n in range(7, N - 1, 14):
+        _, cso = run_oracle(orc, synth.frames(1, n, 1, C, H, W, "uniform"))
+        assert got[n] == cso[0], n
+    del x, z
+    torch.cuda.empty_cache()
 
 
 def test_host_streamed_matches_device(orc):
