@@ -4,12 +4,12 @@ NVCC      ?= /usr/local/cuda/bin/nvcc
 PKG       := paper_conf_ipps_guortgbs11_b200
 CSRC      := $(wildcard $(PKG)/csrc/*.cu)
 CHDR      := $(wildcard $(PKG)/csrc/*.h $(PKG)/csrc/*.cuh) include/aol.h
-BUILD     := build
+BUILD     ?= build
 OBJS      := $(patsubst $(PKG)/csrc/%.cu,$(BUILD)/%.o,$(CSRC))
-LIB       := $(PKG)/libaol.so
+LIB       ?= $(PKG)/libaol.so
 ARCH      := -gencode arch=compute_100a,code=sm_100a
 NVFLAGS   := $(ARCH) -O3 -lineinfo -std=c++17 -Xcompiler -fPIC,-fvisibility=hidden -Xptxas -v \
-             --expt-relaxed-constexpr
+             --expt-relaxed-constexpr $(EXTRA)
 ORACLE    := oracle/liboracle.so
 
 EXAMPLE   := $(BUILD)/aol_example

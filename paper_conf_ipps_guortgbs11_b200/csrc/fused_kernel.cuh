@@ -25,10 +25,12 @@
 //    copies of the contiguous 3-row triple (same smem layout either way).
 //  * Consumer thread r owns repetition r (8 input columns -> 3 Y columns).
 //    int32: two conflict-free LDS.128 per row (the 128B swizzle spreads the
-//    32-byte per-thread stride over all banks).  uint8: one LDS.64 per row and
-//    six DP4A byte-dot-products form the three 6-tap sums.  Either way ONE
-//    warp shuffle supplies the 3-column pattern overlap (pattern {11} vs paving
-//    step 8); lane 31 and the row-wrapping repetition read it from smem.
+//    32-byte per-thread stride over all banks); ONE warp shuffle supplies the
+//    3-column pattern overlap (pattern {11} vs paving step 8), lane 31 and the
+//    row-wrapping repetition read it from smem.  uint8: one LDS.64 per row plus
+//    one LDS.32 of the neighbour's first word (cheaper than shuffle + predicated
+//    load in this issue-bound variant); six DP4A byte-dot-products form the
+//    three 6-tap sums.
 //  * The V stage is a running register accumulation over the band's rows
 //    (4 outputs x 3 columns per thread), so every input row is read once.
 //  * Each finished band (4 output rows, contiguous in Z) is staged in smem and
@@ -67,6 +69,15 @@ __device__ __forceinline__ int32_t task_T(int32_t S) {
 // there without 32-bit overflow (43691 = (2^18 + 2) / 6; checked exhaustively in tests/test_abi.py).
 __device__ __forceinline__ int32_t task_T_nonneg(int32_t S) {
     const int32_t q = int32_t((uint32_t(S) * 43691u) >> 18);
+    return 7 * q - S;
+}
+
+// Same for |S| < 49152 of either sign (V-stage sums of 8-bit-sample frames lie in [-30, 1530]): the
+// arithmetic shift floors S/6 - S/(3*2^18) (= floor(S/6) for S >= 0, = ceil(S/6) - 1 for S < 0, including
+// multiples of 6), so adding the sign bit gives C's truncating S/6 without a multiply-high (IMAD.HI
+// measured slower than IMAD + SHF in this issue-bound kernel; checked exhaustively in tests/test_abi.py).
+__device__ __forceinline__ int32_t task_T_small(int32_t S) {
+    const int32_t q = ((S * 43691) >> 18) + int32_t(uint32_t(S) >> 31);
     return 7 * q - S;
 }
 
@@ -142,8 +153,9 @@ __device__ __forceinline__ void h_row(uint32_t row_base, uint32_t rr, const RepG
         // bytes of x selected by the 0/1 bytes of m (byte k = bits 8k..8k+7 = column 8r+k).
         const uint32_t rowa = row_base + rr * W;
         const uint2 v = ptx::lds64(rowa + g.off0);
-        uint32_t nw = __shfl_down_sync(0xffffffffu, v.x, 1);
-        ptx::lds32_if(nw, rowa + g.offn, g.fix);   // lane 31 / wrapping repetition (predicated)
+        // the neighbour repetition's first word (columns 8r+8..8r+11; word 0 for the row-wrapping repetition):
+        // a second LDS is cheaper here than a shuffle plus the predicated load lane 31 would need
+        const uint32_t nw = ptx::lds32(rowa + g.offn);
         const int32_t S0 = int32_t(__dp4a(v.x, 0x01010101u, __dp4a(v.y, 0x00000101u, 0u)));  // cols 0..5
         const int32_t S1 = int32_t(__dp4a(v.x, 0x01010000u, __dp4a(v.y, 0x01010101u, 0u)));  // cols 2..7
         const int32_t S2 = int32_t(__dp4a(v.y, 0x01010100u, __dp4a(nw, 0x00010101u, 0u)));   // cols 5..10
@@ -263,10 +275,17 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
             int32_t z[4][3];
 #pragma unroll
             for (int m = 0; m < 3; ++m) {
-                z[0][m] = task_T(A0[m]);
-                z[1][m] = task_T(A1[m]);
-                z[2][m] = task_T(A2[m] + add9[m]);
-                z[3][m] = task_T(A3[m] + add911[m]);
+                if constexpr (kI32) {
+                    z[0][m] = task_T(A0[m]);
+                    z[1][m] = task_T(A1[m]);
+                    z[2][m] = task_T(A2[m] + add9[m]);
+                    z[3][m] = task_T(A3[m] + add911[m]);
+                } else {   // 8-bit samples: V sums in [-30, 1530]
+                    z[0][m] = task_T_small(A0[m]);
+                    z[1][m] = task_T_small(A1[m]);
+                    z[2][m] = task_T_small(A2[m] + add9[m]);
+                    z[3][m] = task_T_small(A3[m] + add911[m]);
+                }
             }
             if (tid == 0) ptx::bulk_wait_read<kOutBufs - 1>();   // the out buffer we reuse is free again
             ptx::named_bar_sync(1, NC);

@@ -205,6 +205,11 @@ def test_kernel_division_identities():
     assert np.array_equal(q - np.fmod(S, 6), 7 * q - S)
     U = np.arange(0, 98304, dtype=np.uint64)
     assert np.array_equal(((U * np.uint64(43691)) & np.uint64(0xFFFFFFFF)) >> np.uint64(18), U // np.uint64(6))
+    # signed form for |S| < 49152 (uint8-frame V sums): ((S * 43691) >> 18) + (S < 0), arithmetic shift, in int32
+    T = np.arange(-49151, 49152, dtype=np.int64)
+    p = T * 43691
+    assert p.min() > -(1 << 31) and p.max() < (1 << 31)
+    assert np.array_equal((p >> 18) + (T < 0), np.trunc(T / 6).astype(np.int64))
 
 
 def test_c_example_builds_against_header():
