@@ -57,6 +57,7 @@ int kernel_occupancy(const void* fn, int block, int smem);  // resident CTAs per
 struct FusedPlan {
     int kernel;  // 1 = TMA fused, 2 = generic fused
     int grid, block, smem, stages, bands_per_unit, ctas_per_sm, num_sms, units_per_plane, flags;
+    int reps_per_thread;  // kernel 1: H-tiler repetitions per consumer thread (1, or 2 for wide uint8 frames)
     int64_t units;
 };
 

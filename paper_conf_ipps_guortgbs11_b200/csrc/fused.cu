@@ -48,8 +48,8 @@ bool tma_shape_ok(aol_dtype_t dt, int64_t planes, int64_t channels, int64_t H, i
     return false;
 }
 
-KernelFn pick(aol_dtype_t dt, bool checksum, int block, int cps) {
-    return dt == AOL_U8 ? tma_kernel_u8(checksum, block, cps) : tma_kernel_i32(checksum, block, cps);
+KernelFn pick(aol_dtype_t dt, bool checksum, int kr, int block, int cps) {
+    return dt == AOL_U8 ? tma_kernel_u8(checksum, kr, block, cps) : tma_kernel_i32(checksum, block, cps);
 }
 
 // Shared-memory geometry of the TMA ring: one stage = one row triple.
@@ -112,16 +112,22 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, const void* d_in, const int32_t* d
     bool tma_ok = tma_shape_ok(in_dtype, planes, channels, H, W) && (d_in == nullptr || aligned16(d_in)) &&
                   (d_out == nullptr || aligned16(d_out));
     const RingGeom geom = ring_geom(in_dtype, W);
-    const int nc = int(((W / 8) + 31) / 32 * 32);
+    // repetitions per consumer thread: 2 for uint8 frames at least 1024 wide (HD: 0.498 vs 0.520 ms; 4K: equal),
+    // 1 for narrower ones (CIF: 0.361 vs 0.315 ms -- one half-idle warp per CTA) and for int32
+    // (profiles/r01_u8_r2_ab.jsonl)
+    const int kr = (in_dtype == AOL_U8 && W >= 1024 && !(o.flags & AOL_FLAG_U8_ONE_REP)) ? 2 : 1;
+    const int nc = int(((W / 8 / kr) + 31) / 32 * 32);
     const int block = nc + 32;
     int stages = 0, cps = 1;
     if (tma_ok) {
         // CTAs per SM: enough consumer warps to hide the per-row dependency chains (narrow frames
-        // such as CIF have only 2 consumer warps per CTA), unless the caller fixed it.  The int32
-        // path is HBM-bound with 8 consumer warps per SM; the uint8 path moves 4x fewer input bytes
-        // per row, is issue-bound, and gains from 16 (measured: profiles/r01_u8_*).
+        // such as CIF have only 2 consumer warps per CTA), unless the caller fixed it, but no more
+        // concurrent row streams than that: DRAM efficiency falls as streams are added.  int32
+        // (HBM-bound): 8 consumer warps per SM.  uint8 (issue-bound): 16 warps of one repetition each,
+        // or 8 warps of two (HD: 2 CTAs/SM, 0.499 ms vs 0.567 at 3 and 0.738 at 1;
+        // profiles/r01_u8_r2_ab.jsonl).
         const int cwarps = nc / 32;
-        const int want_warps = in_dtype == AOL_U8 ? 16 : 8;
+        const int want_warps = (in_dtype == AOL_U8 && kr == 1) ? 16 : 8;
         cps = o.ctas_per_sm > 0 ? o.ctas_per_sm
                                 : std::max(1, std::min(8, (want_warps + cwarps - 1) / cwarps));
         for (;; --cps) {
@@ -137,7 +143,7 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, const void* d_in, const int32_t* d
             int occ = 0;
             const int smem = smem_bytes(geom, stages);
             if (stages >= 2 && cps > 1)
-                occ = kernel_occupancy(reinterpret_cast<const void*>(pick(in_dtype, true, block, cps)), block, smem);
+                occ = kernel_occupancy(reinterpret_cast<const void*>(pick(in_dtype, true, kr, block, cps)), block, smem);
             if (cps == 1) occ = 1;   // one CTA always fits once its shared memory does
             if ((stages >= 2 && occ >= cps) || cps == 1 || o.ctas_per_sm > 0) {
                 if (stages < 2) tma_ok = false;
@@ -180,6 +186,7 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, const void* d_in, const int32_t* d
         plan->stages = stages;
         plan->smem = smem_bytes(geom, stages);
         plan->ctas_per_sm = cps;
+        plan->reps_per_thread = kr;
         plan->flags = o.flags;
     } else {
         plan->kernel = 2;
@@ -250,7 +257,7 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
     a.hint_stores = (plan.flags & AOL_FLAG_EVICT_FIRST_STORES) ? 1 : 0;
     a.blocked_units = (plan.flags & AOL_FLAG_BLOCKED_UNITS) ? 1 : 0;
 
-    KernelFn k = pick(in_dtype, d_cs != nullptr, plan.block, plan.ctas_per_sm);
+    KernelFn k = pick(in_dtype, d_cs != nullptr, plan.reps_per_thread, plan.block, plan.ctas_per_sm);
     aol_status_t st_attr = kernel_smem(reinterpret_cast<const void*>(k), plan.smem);
     if (st_attr != AOL_OK) return st_attr;
     k<<<grid, plan.block, plan.smem, s>>>(map, a);

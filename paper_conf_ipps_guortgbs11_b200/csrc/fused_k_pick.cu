@@ -7,11 +7,14 @@ KernelFn tma_kernel_i32_cs(int block, int cps);
 KernelFn tma_kernel_i32_nocs(int block, int cps);
 KernelFn tma_kernel_u8_cs(int block, int cps);
 KernelFn tma_kernel_u8_nocs(int block, int cps);
+KernelFn tma_kernel_u8r2_cs(int block, int cps);
+KernelFn tma_kernel_u8r2_nocs(int block, int cps);
 
 KernelFn tma_kernel_i32(bool checksum, int block, int cps) {
     return checksum ? tma_kernel_i32_cs(block, cps) : tma_kernel_i32_nocs(block, cps);
 }
-KernelFn tma_kernel_u8(bool checksum, int block, int cps) {
+KernelFn tma_kernel_u8(bool checksum, int reps_per_thread, int block, int cps) {
+    if (reps_per_thread == 2) return checksum ? tma_kernel_u8r2_cs(block, cps) : tma_kernel_u8r2_nocs(block, cps);
     return checksum ? tma_kernel_u8_cs(block, cps) : tma_kernel_u8_nocs(block, cps);
 }
 }  // namespace fused

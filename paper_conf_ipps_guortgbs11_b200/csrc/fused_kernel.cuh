@@ -127,11 +127,13 @@ struct RepGeom {
     bool fix;             // read the neighbour from smem instead of the shuffle
 };
 
-// H stage of one input row: the three 6-tap window sums of repetition r, T() applied.
-template <typename Tin>
+// H stage of one input row: the three 6-tap window sums of each of the thread's kR repetitions, T() applied:
+// y[3j + k] = T(window k of repetition j).
+template <typename Tin, int kR>
 __device__ __forceinline__ void h_row(uint32_t row_base, uint32_t rr, const RepGeom& g, uint32_t segs, uint32_t W,
-                                      int32_t& y0, int32_t& y1, int32_t& y2) {
+                                      int32_t (&y)[3 * kR]) {
     if constexpr (std::is_same<Tin, int32_t>::value) {
+        static_assert(kR == 1, "int32 path: one repetition per thread");
         const uint32_t line = rr * segs + g.seg;
         const int4 q0 = ptx::lds128(row_base + swz(line, g.off0));
         const int4 q1 = ptx::lds128(row_base + swz(line, g.off1));
@@ -145,30 +147,49 @@ __device__ __forceinline__ void h_row(uint32_t row_base, uint32_t rr, const RepG
         int4 qn = q0;   // lane 31 / wrapping repetition: neighbour chunk from smem (predicated, no branch)
         ptx::lds128_if(qn, row_base + swz(rr * segs + g.segn, g.offn), g.fix);
         dn = g.fix ? qn.x + qn.y + qn.z : dn;
-        y0 = task_T(e + qp);            // window cols 0..5
-        y1 = task_T(qp + f);            // window cols 2..7
-        y2 = task_T(q1.y + f + dn);     // window cols 5..10
+        y[0] = task_T(e + qp);            // window cols 0..5
+        y[1] = task_T(qp + f);            // window cols 2..7
+        y[2] = task_T(q1.y + f + dn);     // window cols 5..10
     } else {
-        // uint8 samples: bytes 0..7 of the repetition in two words; dp4a(x, m, c) = c + sum of the
-        // bytes of x selected by the 0/1 bytes of m (byte k = bits 8k..8k+7 = column 8r+k).
+        // uint8 samples: the kR repetitions' 8*kR bytes in 2*kR words, then the next repetition's first word
+        // (columns 8(r+kR)..; word 0 for the row-wrapping repetition); dp4a(x, m, c) = c + sum of the bytes
+        // of x selected by the 0/1 bytes of m (byte k = bits 8k..8k+7 = column 8r+k).
         const uint32_t rowa = row_base + rr * W;
-        const uint2 v = ptx::lds64(rowa + g.off0);
-        // the neighbour repetition's first word (columns 8r+8..8r+11; word 0 for the row-wrapping repetition):
-        // a second LDS is cheaper here than a shuffle plus the predicated load lane 31 would need
-        const uint32_t nw = ptx::lds32(rowa + g.offn);
-        const int32_t S0 = int32_t(__dp4a(v.x, 0x01010101u, __dp4a(v.y, 0x00000101u, 0u)));  // cols 0..5
-        const int32_t S1 = int32_t(__dp4a(v.x, 0x01010000u, __dp4a(v.y, 0x01010101u, 0u)));  // cols 2..7
-        const int32_t S2 = int32_t(__dp4a(v.y, 0x01010100u, __dp4a(nw, 0x00010101u, 0u)));   // cols 5..10
-        y0 = task_T_nonneg(S0);   // 8-bit samples: 0 <= S <= 1530
-        y1 = task_T_nonneg(S1);
-        y2 = task_T_nonneg(S2);
+        uint32_t x[2 * kR + 1];
+        if constexpr (kR == 1) {
+            const uint2 v = ptx::lds64(rowa + g.off0);
+            x[0] = v.x;
+            x[1] = v.y;
+        } else {
+            static_assert(kR == 2, "uint8 path: 1 or 2 repetitions per thread");
+            const int4 v = ptx::lds128(rowa + g.off0);
+            x[0] = uint32_t(v.x);
+            x[1] = uint32_t(v.y);
+            x[2] = uint32_t(v.z);
+            x[3] = uint32_t(v.w);
+        }
+        x[2 * kR] = ptx::lds32(rowa + g.offn);
+#pragma unroll
+        for (int j = 0; j < kR; ++j) {
+            const uint32_t lo = x[2 * j], hi = x[2 * j + 1], nw = x[2 * j + 2];
+            const int32_t S0 = int32_t(__dp4a(lo, 0x01010101u, __dp4a(hi, 0x00000101u, 0u)));  // cols 0..5
+            const int32_t S1 = int32_t(__dp4a(lo, 0x01010000u, __dp4a(hi, 0x01010101u, 0u)));  // cols 2..7
+            const int32_t S2 = int32_t(__dp4a(hi, 0x01010100u, __dp4a(nw, 0x00010101u, 0u)));  // cols 5..10
+            y[3 * j + 0] = task_T_nonneg(S0);   // 8-bit samples: 0 <= S <= 1530
+            y[3 * j + 1] = task_T_nonneg(S1);
+            y[3 * j + 2] = task_T_nonneg(S2);
+        }
     }
 }
 
-template <typename Tin, bool kChecksum, int kMaxThreads, int kMinBlocks>
+// kR = repetitions of the H tiler per consumer thread: 1 for int32 (two LDS.128 already cover one repetition's
+// 8 columns); 1 or 2 for uint8 input, whose 16 bytes for two repetitions come in one LDS.128 and whose per-stage
+// bookkeeping (mbarrier wait/arrive, addressing) two repetitions then share (the host picks, fused.cu).
+template <typename Tin, int kR, bool kChecksum, int kMaxThreads, int kMinBlocks>
 __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
     fused_tma_kernel(const __grid_constant__ CUtensorMap tmap, const FusedArgs a) {
     constexpr bool kI32 = std::is_same<Tin, int32_t>::value;
+    constexpr int kC = 3 * kR;   // Y / Z columns per consumer thread
     extern __shared__ uint8_t smem_raw[];
     uint8_t* smem = reinterpret_cast<uint8_t*>((reinterpret_cast<uintptr_t>(smem_raw) + 1023) & ~uintptr_t(1023));
     uint8_t* stage_base = smem;
@@ -232,9 +253,9 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
 
     // ---------------------------------------------------- consumer threads
     const int lane = tid & 31;
-    const bool active = tid < a.reps;
-    const int r = active ? tid : a.reps - 1;        // repetition owned (clamped for idle lanes)
-    const int rn = (r + 1 == a.reps) ? 0 : r + 1;  // neighbour repetition (toroidal, Fig. 11 '% 1920')
+    const bool active = kR * tid < a.reps;
+    const int r = active ? kR * tid : a.reps - kR;   // first repetition owned (clamped for idle lanes)
+    const int rn = (r + kR == a.reps) ? 0 : r + kR;  // next thread's repetition (toroidal, Fig. 11 '% 1920')
     RepGeom g;
     g.fix = (lane == 31) || (r + 1 == a.reps);
     if constexpr (kI32) {
@@ -248,6 +269,7 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
         g.off0 = 8u * uint32_t(r);
         g.off1 = g.off0 + 4;
         g.offn = 8u * uint32_t(rn);
+        g.fix = false;
     }
     const uint32_t segs = uint32_t(a.segs);
     const uint32_t Wu = uint32_t(a.W);
@@ -265,16 +287,16 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
         const int32_t chan = int32_t(plane % a.channels);
         uint64_t csacc = 0;
 
-        int32_t A0[3], A1[3], A2[3], A3[3];   // running V window sums of the current band
-        int32_t Hr9[3], Hr911[3];             // halo: Y row 9 and rows 9..11 of the unit's last band
+        int32_t A0[kC], A1[kC], A2[kC], A3[kC];   // running V window sums of the current band
+        int32_t Hr9[kC], Hr911[kC];               // halo: Y row 9 and rows 9..11 of the unit's last band
 #pragma unroll
-        for (int m = 0; m < 3; ++m) A0[m] = A1[m] = A2[m] = A3[m] = Hr9[m] = Hr911[m] = 0;
+        for (int m = 0; m < kC; ++m) A0[m] = A1[m] = A2[m] = A3[m] = Hr9[m] = Hr911[m] = 0;
 
         // Band `band` is complete once rows 9..11 of its pattern are known: z = T(window sums).
         auto emit = [&](int32_t band, const int32_t* add9, const int32_t* add911) {
-            int32_t z[4][3];
+            int32_t z[4][kC];
 #pragma unroll
-            for (int m = 0; m < 3; ++m) {
+            for (int m = 0; m < kC; ++m) {
                 if constexpr (kI32) {
                     z[0][m] = task_T(A0[m]);
                     z[1][m] = task_T(A1[m]);
@@ -294,7 +316,14 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
 #pragma unroll
                 for (int k = 0; k < 4; ++k)
 #pragma unroll
-                    for (int m = 0; m < 3; ++m) ptx::sts32(ob + 4u * uint32_t(k * Wo + 3 * r + m), z[k][m]);
+                    if constexpr (kR == 1) {
+#pragma unroll
+                        for (int m = 0; m < 3; ++m) ptx::sts32(ob + 4u * uint32_t(k * Wo + 3 * r + m), z[k][m]);
+                    } else {   // 8-byte aligned pairs: Wo = 6 (W/16) and 3r are even
+#pragma unroll
+                        for (int m = 0; m < kC; m += 2)
+                            ptx::sts64(ob + 4u * uint32_t(k * Wo + 3 * r + m), z[k][m], z[k][m + 1]);
+                    }
             }
             ptx::fence_proxy_async_smem();
             ptx::named_bar_sync(1, NC);
@@ -316,13 +345,13 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
 #pragma unroll
                 for (int k = 0; k < 4; ++k)
 #pragma unroll
-                    for (int m = 0; m < 3; ++m)
+                    for (int m = 0; m < kC; ++m)
                         csacc += uint64_t(uint32_t(z[k][m])) * uint64_t(w0 + uint32_t(k * Wo + m));
             }
         };
 
         // Wait for the next ring stage, run the H stage on its 3 rows (y[row][col]), release the stage.
-        auto triple = [&](int32_t (&y)[3][3]) {
+        auto triple = [&](int32_t (&y)[3][kC]) {
             ptx::mbar_wait_sleep(&full[s], ph);
             const uint32_t sb = stage_s32 + uint32_t(s) * a.stage_stride;   // 32-bit shared address
 #pragma unroll
@@ -330,9 +359,10 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
 #ifdef AOL_PROBE_STREAM_ONLY
                 // measurement build only (tools/stream_probe.sh): skip the smem reads and H arithmetic to
                 // expose the pure TMA streaming rate of this access pattern.  Never in libaol.so.
-                y[rr][0] = y[rr][1] = y[rr][2] = int32_t(sb) + rr;
+#pragma unroll
+                for (int m = 0; m < kC; ++m) y[rr][m] = int32_t(sb) + rr;
 #else
-                h_row<Tin>(sb, uint32_t(rr), g, segs, Wu, y[rr][0], y[rr][1], y[rr][2]);
+                h_row<Tin, kR>(sb, uint32_t(rr), g, segs, Wu, y[rr]);
 #endif
             }
             __syncwarp();
@@ -344,36 +374,36 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
         };
 
         {   // the halo triple comes first: keep what the unit's last band needs from it (rows 9 and 9..11)
-            int32_t y[3][3];
+            int32_t y[3][kC];
             triple(y);
 #pragma unroll
-            for (int m = 0; m < 3; ++m) {
+            for (int m = 0; m < kC; ++m) {
                 Hr9[m] = y[0][m];
                 Hr911[m] = y[0][m] + y[1][m] + y[2][m];
             }
         }
         // ---- one band per iteration; V stage = running sums of the 12-row pattern (windows at rows 0,2,4,6)
         for (int32_t band = b0; band < b1; ++band) {
-            int32_t y[3][3];
+            int32_t y[3][kC];
             triple(y);   // rows 0..2
             if (band > b0) {
                 // rows 0..2 of this band are rows 9..11 of the previous one: emit it
-                int32_t r9[3], r911[3];
+                int32_t r9[kC], r911[kC];
 #pragma unroll
-                for (int m = 0; m < 3; ++m) {
+                for (int m = 0; m < kC; ++m) {
                     r9[m] = y[0][m];
                     r911[m] = y[0][m] + y[1][m] + y[2][m];
                 }
                 emit(band - 1, r9, r911);
             }
 #pragma unroll
-            for (int m = 0; m < 3; ++m) {
+            for (int m = 0; m < kC; ++m) {
                 A0[m] = y[0][m] + y[1][m] + y[2][m];   // rows 0..2 of window 0..5
                 A1[m] = y[2][m];                        // row 2 of window 2..7
             }
             triple(y);   // rows 3..5
 #pragma unroll
-            for (int m = 0; m < 3; ++m) {
+            for (int m = 0; m < kC; ++m) {
                 const int32_t s3 = y[0][m] + y[1][m] + y[2][m];
                 A0[m] += s3;
                 A1[m] += s3;
@@ -381,7 +411,7 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
             }
             triple(y);   // rows 6..8
 #pragma unroll
-            for (int m = 0; m < 3; ++m) {
+            for (int m = 0; m < kC; ++m) {
                 const int32_t s2 = y[0][m] + y[1][m];
                 A1[m] += s2;
                 A2[m] += s2 + y[2][m];
@@ -486,15 +516,23 @@ using KernelFn = void (*)(const CUtensorMap, const FusedArgs);
 
 // Explicit instantiations live in fused_k_*.cu (compiled in parallel); these pick one.
 KernelFn tma_kernel_i32(bool checksum, int block, int cps);
-KernelFn tma_kernel_u8(bool checksum, int block, int cps);
+KernelFn tma_kernel_u8(bool checksum, int reps_per_thread, int block, int cps);
 
-template <typename Tin, bool kChecksum>
+template <typename Tin, int kR, bool kChecksum>
 KernelFn pick_tma_kernel(int block, int cps) {
-    if (block <= 128 && cps >= 3) return fused_tma_kernel<Tin, kChecksum, 128, 4>;
-    if (block <= 320 && cps >= 3) return fused_tma_kernel<Tin, kChecksum, 320, 3>;
-    if (block <= 320 && cps >= 2) return fused_tma_kernel<Tin, kChecksum, 320, 2>;
-    if (block <= 512) return fused_tma_kernel<Tin, kChecksum, 512, 1>;
-    return fused_tma_kernel<Tin, kChecksum, 1024, 1>;
+    if constexpr (kR == 2) {
+        // two repetitions per thread take ~126 registers: bounds that never force spills below 1024 threads
+        if (block <= 160 && cps >= 3) return fused_tma_kernel<Tin, kR, kChecksum, 160, 3>;
+        if (block <= 256 && cps >= 2) return fused_tma_kernel<Tin, kR, kChecksum, 256, 2>;
+        if (block <= 512) return fused_tma_kernel<Tin, kR, kChecksum, 512, 1>;
+        return fused_tma_kernel<Tin, kR, kChecksum, 1024, 1>;
+    } else {
+        if (block <= 128 && cps >= 3) return fused_tma_kernel<Tin, kR, kChecksum, 128, 4>;
+        if (block <= 320 && cps >= 3) return fused_tma_kernel<Tin, kR, kChecksum, 320, 3>;
+        if (block <= 320 && cps >= 2) return fused_tma_kernel<Tin, kR, kChecksum, 320, 2>;
+        if (block <= 512) return fused_tma_kernel<Tin, kR, kChecksum, 512, 1>;
+        return fused_tma_kernel<Tin, kR, kChecksum, 1024, 1>;
+    }
 }
 
 }  // namespace fused

@@ -69,6 +69,10 @@ __device__ __forceinline__ void sts32(uint32_t saddr, int32_t v) {
     asm volatile("st.shared.s32 [%0], %1;" ::"r"(saddr), "r"(v) : "memory");
 }
 
+__device__ __forceinline__ void sts64(uint32_t saddr, int32_t a, int32_t b) {
+    asm volatile("st.shared.v2.s32 [%0], {%1, %2};" ::"r"(saddr), "r"(a), "r"(b) : "memory");
+}
+
 // Predicated 32-bit / 128-bit shared loads (no branch): v is left unchanged when !pred.
 __device__ __forceinline__ void lds32_if(uint32_t& v, uint32_t saddr, bool pred) {
     asm volatile("{\n\t.reg .pred p;\n\tsetp.ne.b32 p, %2, 0;\n\t@p ld.shared.u32 %0, [%1];\n\t}"

@@ -145,6 +145,31 @@ def test_fused_u8_launch_options(orc):
         assert np.array_equal(np_u64(cs), cso), o
 
 
+@pytest.mark.parametrize("W", [1024, 1040, 1920, 2048, 3968])
+def test_fused_u8_two_reps_per_thread(orc, W):
+    """uint8 frames >= 1024 wide run two H repetitions per consumer thread (one LDS.128 for 16 samples);
+    AOL_FLAG_U8_ONE_REP (32) forces one.  Both against the oracle, incl. W % 128 != 0 (1-D bulk copies),
+    warps with idle lanes (W = 1040: 65 threads) and the row-wrapping repetition pair; with and without
+    the checksum epilogue."""
+    N, C, H = 2, 3, 36
+    xh = synth.frames(23, 0, N, C, H, W, "uniform")
+    xh[0, 1] = synth.frames(24, 0, 1, 1, H, W, "dark")[0, 0]   # negative V sums on one plane
+    zo, cso = run_oracle(orc, xh)
+    x8 = torch.from_numpy(xh.astype(np.uint8)).cuda()
+    for flags in (0, 32, 16):
+        o = {"kernel": 1, "flags": flags}
+        plan = aol.downscale_frame_plan(N, C, H, W, dtype=torch.uint8, opts=o)
+        z, cs = aol.downscale_frame(x8, checksums=True, opts=o)
+        z2, _ = aol.downscale_frame(x8, opts=o)
+        torch.cuda.synchronize()
+        assert np.array_equal(z.cpu().numpy(), zo), flags
+        assert np.array_equal(z2.cpu().numpy(), zo), flags
+        assert np.array_equal(np_u64(cs), cso), flags
+        # block = consumer threads (W/8 repetitions / reps-per-thread, whole warps) + 1 producer warp
+        kr = 1 if flags == 32 else 2
+        assert plan["block"] == ((W // 8 // kr) + 31) // 32 * 32 + 32, (flags, plan)
+
+
 def test_no_checksum_and_zero_frames(orc):
     xh = synth.frames(1, 0, 1, 3, 18, 64)
     z, cs = aol.downscale_frame(torch.from_numpy(xh).cuda())
