@@ -367,7 +367,8 @@ def main():
                      "traffic": traffic, "peak_source": peak_src,
                      "algorithmic_bytes_per_launch": bpf * calls[0],
                      "avg_launch_ms": avg_launch_s * 1000.0, "min_launch_ms": min(launch_ms)},
-        "gpu_launches": a.steps * len(calls),
+        # per call: zero_checksums_kernel + the fused kernel (its programmatic dependent)
+        "gpu_launches": a.steps * len(calls) * (2 if plan["kernel"] == 1 else 1),
         "clocks": clk.summary(),
     }
     if e2e is not None:

@@ -113,6 +113,8 @@ typedef struct {
 #define AOL_FLAG_BLOCKED_UNITS 8       /* each CTA takes a contiguous block of work units (default:
                                           round-robin, so concurrently running CTAs are adjacent)  */
 #define AOL_FLAG_U8_BULK 16            /* uint8 input: 1-D bulk copies even when W % 128 == 0      */
+#define AOL_FLAG_NO_PDL 64             /* launch the fused kernel after the checksum zeroing completes
+                                          (default: overlapped, programmatic dependent launch)        */
 #define AOL_FLAG_U8_ONE_REP 32         /* uint8 input: one H repetition per consumer thread even for
                                           W >= 1024 (default there: two)                            */
 

@@ -16,6 +16,14 @@ using namespace fused;
 
 namespace {
 
+// Zeroes the per-frame checksums ahead of a fused launch.  It lets that launch start at once
+// (griddepcontrol.launch_dependents): the fused kernel's prologue, TMA ring fill and whole first work unit
+// overlap this kernel, and only its first checksum atomic waits for it (ptx::griddep_wait).
+__global__ void __launch_bounds__(256) zero_checksums_kernel(uint64_t* __restrict__ cs, int64_t n) {
+    ptx::griddep_launch_dependents();
+    for (int64_t i = threadIdx.x; i < n; i += blockDim.x) cs[i] = 0;
+}
+
 // ------------------------------------------------------------ TMA descriptor
 using EncodeTiledFn = CUresult (*)(CUtensorMap*, CUtensorMapDataType, cuuint32_t, void*, const cuuint64_t*,
                                    const cuuint64_t*, const cuuint32_t*, const cuuint32_t*, CUtensorMapInterleave,
@@ -184,7 +192,10 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, const void* d_in, const int32_t* d
         plan->grid = int(std::min<int64_t>(plan->units, max_ctas));
         plan->block = block;
         plan->stages = stages;
-        plan->smem = smem_bytes(geom, stages);
+        // The grid is persistent (cps CTAs per SM, units assigned round-robin): pad the shared memory so
+        // that no SM can take a (cps+1)-th CTA, which would leave another SM short and stretch the tail.
+        const int exclusive = dev.smem_per_sm / (cps + 1) - 1024 + 128;
+        plan->smem = std::max(smem_bytes(geom, stages), std::min(exclusive, dev.smem_optin));
         plan->ctas_per_sm = cps;
         plan->reps_per_thread = kr;
         plan->flags = o.flags;
@@ -203,9 +214,9 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
                           int64_t frames, int64_t channels, int64_t H, int64_t W, uint64_t* d_cs, cudaStream_t s) {
     const int64_t planes = frames * channels;
     const int32_t Ho = int32_t(4 * (H / 9)), Wo = int32_t(3 * (W / 8));
-    if (d_cs) AOL_CUDA_TRY(cudaMemsetAsync(d_cs, 0, size_t(frames) * sizeof(uint64_t), s));
 
     if (plan.kernel == 2) {
+        if (d_cs) AOL_CUDA_TRY(cudaMemsetAsync(d_cs, 0, size_t(frames) * sizeof(uint64_t), s));
         if (in_dtype == AOL_U8) {
             auto k = d_cs ? fused_generic_kernel<uint8_t, true> : fused_generic_kernel<uint8_t, false>;
             k<<<plan.grid, plan.block, 0, s>>>(static_cast<const uint8_t*>(d_in), d_out, d_cs, planes, int32_t(H),
@@ -260,7 +271,30 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
     KernelFn k = pick(in_dtype, d_cs != nullptr, plan.reps_per_thread, plan.block, plan.ctas_per_sm);
     aol_status_t st_attr = kernel_smem(reinterpret_cast<const void*>(k), plan.smem);
     if (st_attr != AOL_OK) return st_attr;
-    k<<<grid, plan.block, plan.smem, s>>>(map, a);
+    // With checksums: zero them in a one-CTA kernel and launch the fused kernel as its programmatic
+    // dependent, so the zeroing (and the launch gap after it) overlaps the fused kernel's start instead of
+    // preceding it (single-frame latency).  Only the zero kernel can be the primary: it
+    // is an ordinary launch, so everything earlier in the stream (e.g. the producer of X) has completed.
+    if (d_cs) {
+        zero_checksums_kernel<<<1, 256, 0, s>>>(d_cs, frames);
+        AOL_LAUNCH_CHECK("zero_checksums_kernel");
+    }
+    cudaLaunchConfig_t cfg;
+    std::memset(&cfg, 0, sizeof cfg);
+    cfg.gridDim = dim3(unsigned(grid));
+    cfg.blockDim = dim3(unsigned(plan.block));
+    cfg.dynamicSmemBytes = size_t(plan.smem);
+    cfg.stream = s;
+    cudaLaunchAttribute attr[1];
+    attr[0].id = cudaLaunchAttributeProgrammaticStreamSerialization;
+    attr[0].val.programmaticStreamSerializationAllowed = 1;
+    cfg.attrs = attr;
+    cfg.numAttrs = (d_cs && !(plan.flags & AOL_FLAG_NO_PDL)) ? 1 : 0;
+    cudaError_t le = cudaLaunchKernelEx(&cfg, k, map, a);
+    if (le != cudaSuccess) {
+        set_error("launch of fused_tma_kernel failed: %s", cudaGetErrorString(le));
+        return AOL_E_CUDA;
+    }
     AOL_LAUNCH_CHECK("fused_tma_kernel");
     return AOL_OK;
 }

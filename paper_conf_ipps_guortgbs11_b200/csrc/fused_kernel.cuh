@@ -429,6 +429,10 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
             if (tid == 0) {
                 unsigned long long sum = 0;
                 for (int w = 0; w < NC / 32; ++w) sum += red[w];
+                // the checksums were zeroed by the preceding zero_checksums_kernel, which this launch may
+                // overlap (programmatic dependent launch): wait for it before the first atomic (no-op when
+                // the kernel was launched without the PDL attribute, and after the first wait)
+                ptx::griddep_wait();
                 atomicAdd(reinterpret_cast<unsigned long long*>(a.cs + plane / a.channels), sum);
             }
             ptx::named_bar_sync(2, NC);   // red[] is reused by the next unit

@@ -69,6 +69,13 @@ __device__ __forceinline__ void sts32(uint32_t saddr, int32_t v) {
     asm volatile("st.shared.s32 [%0], %1;" ::"r"(saddr), "r"(v) : "memory");
 }
 
+// Programmatic dependent launch: a secondary grid waits for its primary's completion and memory
+// (no-op without the launch attribute); a primary allows its dependents to launch early.
+__device__ __forceinline__ void griddep_wait() { asm volatile("griddepcontrol.wait;" ::: "memory"); }
+__device__ __forceinline__ void griddep_launch_dependents() {
+    asm volatile("griddepcontrol.launch_dependents;" ::: "memory");
+}
+
 __device__ __forceinline__ void sts64(uint32_t saddr, int32_t a, int32_t b) {
     asm volatile("st.shared.v2.s32 [%0], {%1, %2};" ::"r"(saddr), "r"(a), "r"(b) : "memory");
 }

@@ -28,7 +28,7 @@ def test_bench_default_contract():
     d = run("--frames", "12", "--H", "36", "--W", "128", "--steps", "5", "--warmup", "3")
     assert REQUIRED <= set(d)
     assert d["scaling"] == "weak" and d["n_gpus"] == 1 and d["higher_is_better"] is True
-    assert d["value"] > 0 and d["gpu_launches"] == 5 and d["steps"] == 5 and d["warmup"] == 3
+    assert d["value"] > 0 and d["gpu_launches"] == 10 and d["steps"] == 5 and d["warmup"] == 3
     r = d["roofline"]
     assert r["bound"] == "hbm" and r["unit"] == "GB/s" and abs(r["frac"] - r["achieved"] / r["peak"]) < 1e-9
     assert {"value", "unit", "h2d_bytes_per_step", "d2h_bytes_per_step"} <= set(d["e2e"])
@@ -40,7 +40,7 @@ def test_bench_default_contract():
 def test_bench_stream_mode():
     d = run("--stream-frames", "50", "--pool", "16", "--H", "36", "--W", "128", "--steps", "3", "--warmup", "3",
             "--no-cpu-baseline")
-    assert d["scaling"] == "strong" and d["config"]["launches_per_step"] == 4 and d["gpu_launches"] == 12
+    assert d["scaling"] == "strong" and d["config"]["launches_per_step"] == 4 and d["gpu_launches"] == 24
 
 
 def test_bench_reference_arm():
