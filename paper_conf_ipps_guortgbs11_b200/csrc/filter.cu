@@ -16,6 +16,7 @@
 
 #include <algorithm>
 #include <cstdint>
+#include <cstdlib>
 #include <cstring>
 #include <type_traits>
 
@@ -41,7 +42,15 @@ struct FilterDev {
     // extent needs no modulo, and its elements sit at base + lin[p] (row-major element offsets)
     int32_t fmax_in[AOL_MAX_RANK], fmax_out[AOL_MAX_RANK];
     int64_t lin_in[AOL_MAX_FILTER_PATTERN], lin_out[AOL_MAX_WINDOWS];
+    // magic numbers: x mod s_in/s_out (x < 2^31) and |S| / |divisor| (|S| <= 2^31) as (umulhi(x, mul) + x) >> sh
+    uint32_t mi_mul[AOL_MAX_RANK], mi_sh[AOL_MAX_RANK], mo_mul[AOL_MAX_RANK], mo_sh[AOL_MAX_RANK];
+    uint32_t dv_mul, dv_sh;
 };
+
+// floor(x / d) for 0 <= x <= 2^31 and the host-computed (mul, sh) of d (1 <= d < 2^31)
+__device__ __forceinline__ uint32_t udiv_magic(uint32_t x, uint32_t mul, uint32_t sh) {
+    return (__umulhi(x, mul) + x) >> sh;
+}
 
 // D bounds every rank involved (array ranks of both tilers, repetition rank): loops unroll to D.
 template <int D, bool kFast32>
@@ -223,6 +232,150 @@ __global__ void __launch_bounds__(256) filter32_kernel(const FilterDev fd, const
     }
 }
 
+// Register-pattern variant for input patterns of at most 16 elements (the paper's filters: 11 and 12):
+// each pattern element is loaded ONCE per repetition into registers -- four at a time with 128-bit loads
+// when the pattern is a contiguous run of the array (lin_in[p] == p, e.g. the H filter's 11 columns) and
+// the repetition's run is 16-byte aligned -- and every window sum is then formed from registers by a
+// predicated walk over the NP elements (no dynamic register indexing).  The generic kernel above instead
+// issues window_len loads per window (18 for H, 24 for V), most of them L1 hits of a scattered warp access.
+template <int D, int NP>
+__global__ void __launch_bounds__(256) filter32_reg_kernel(const FilterDev fd, const int32_t* __restrict__ in,
+                                                           int32_t* __restrict__ out, int32_t in_elems,
+                                                           int32_t contig) {
+    __shared__ int32_t lin_out[AOL_MAX_WINDOWS], start[AOL_MAX_WINDOWS];
+    // per-thread prefix sums of the pattern, [p][thread] (conflict-free: a warp reads one row at a time)
+    __shared__ int32_t pre[(NP + 1) * 256];
+    if (threadIdx.x < AOL_MAX_WINDOWS) {
+        lin_out[threadIdx.x] = int32_t(fd.lin_out[threadIdx.x]);
+        start[threadIdx.x] = fd.start[threadIdx.x];
+    }
+    __syncthreads();
+    int32_t* my = pre + threadIdx.x;
+    const int32_t nrep = int32_t(fd.nrep);
+    for (int32_t r = int32_t(blockIdx.x * blockDim.x + threadIdx.x); r < nrep; r += int32_t(gridDim.x * blockDim.x)) {
+        int32_t vi[D], vo[D];
+#pragma unroll
+        for (int a = 0; a < D; ++a) {
+            vi[a] = fd.o_in[a];
+            vo[a] = fd.o_out[a];
+        }
+        uint32_t n = uint32_t(r);
+#pragma unroll
+        for (int j = D - 1; j >= 0; --j) {
+            if (j < fd.rr) {
+                const uint32_t q = (__umulhi(n, fd.fd_mul[j]) + n) >> fd.fd_shift[j];
+                const int32_t i = int32_t(n - q * uint32_t(fd.rep_ext[j]));
+                n = q;
+#pragma unroll
+                for (int a = 0; a < D; ++a) {   // reference points o' + P'.r (Section IV)
+                    vi[a] += fd.P_in[a][j] * i;
+                    vo[a] += fd.P_out[a][j] * i;
+                }
+            }
+        }
+        bool in_ok = true, out_ok = true;
+        int32_t base_in = 0, base_out = 0;
+#pragma unroll
+        for (int a = 0; a < D; ++a) {   // mod s (all terms >= 0 and < 2^31): magic-number division
+            if (a < fd.ra_in) {
+                vi[a] -= int32_t(udiv_magic(uint32_t(vi[a]), fd.mi_mul[a], fd.mi_sh[a])) * fd.s_in[a];
+                in_ok &= vi[a] + fd.fmax_in[a] < fd.s_in[a];
+                base_in += vi[a] * int32_t(fd.st_in[a]);
+            }
+            if (a < fd.ra_out) {
+                vo[a] -= int32_t(udiv_magic(uint32_t(vo[a]), fd.mo_mul[a], fd.mo_sh[a])) * fd.s_out[a];
+                out_ok &= vo[a] + fd.fmax_out[a] < fd.s_out[a];
+                base_out += vo[a] * int32_t(fd.st_out[a]);
+            }
+        }
+        // gather (Fig. 4): the repetition's pattern, each element once
+        int32_t x[NP];
+        if (contig && in_ok && (base_in & 3) == 0 && base_in + NP <= in_elems) {
+#pragma unroll
+            for (int v = 0; v < NP / 4; ++v) {
+                const int4 q = __ldg(reinterpret_cast<const int4*>(in + base_in) + v);
+                x[4 * v] = q.x;
+                x[4 * v + 1] = q.y;
+                x[4 * v + 2] = q.z;
+                x[4 * v + 3] = q.w;
+            }
+        } else {
+#pragma unroll
+            for (int p = 0; p < NP; ++p) {
+                x[p] = 0;
+                if (p < fd.n_in) {
+                    int32_t off;
+                    if (in_ok) {
+                        off = base_in + int32_t(fd.lin_in[p]);
+                    } else {
+                        off = 0;
+#pragma unroll
+                        for (int a = 0; a < D; ++a) {
+                            if (a < fd.ra_in) {
+                                int32_t c = vi[a] + fd.f_in[p][a];   // toroidal pattern element
+                                if (c >= fd.s_in[a]) c -= fd.s_in[a];
+                                off += c * int32_t(fd.st_in[a]);
+                            }
+                        }
+                    }
+                    x[p] = __ldg(in + off);
+                }
+            }
+        }
+        // prefix sums: window k's sum = pre[start_k + len] - pre[start_k] (two LDS, whatever the window)
+        {
+            int32_t acc = 0;
+            my[0] = 0;
+#pragma unroll
+            for (int p = 0; p < NP; ++p) {
+                acc += x[p];
+                my[(p + 1) * 256] = acc;
+            }
+        }
+        for (int k = 0; k < fd.n_win; ++k) {
+            // task (Fig. 5): S over window k = elements start_k .. start_k + len - 1, tile = S/d - S%d
+            const int32_t s0 = start[k];
+            const int32_t S = my[(s0 + fd.len) * 256] - my[s0 * 256];
+            // tile = S/d - S%d (C semantics) = q (1 + d) - S with q = trunc(S/d) = sign(S) sign(d) floor(|S|/|d|)
+            const uint32_t qa = udiv_magic(uint32_t(abs(S)), fd.dv_mul, fd.dv_sh);   // |INT_MIN| = 2^31 ok
+            const int32_t q = ((S < 0) != (fd.divisor < 0)) ? -int32_t(qa) : int32_t(qa);
+            const int32_t tile = q * (1 + fd.divisor) - S;
+            int32_t off = base_out + lin_out[k];
+            if (!out_ok) {
+                off = 0;
+#pragma unroll
+                for (int a = 0; a < D; ++a) {
+                    if (a < fd.ra_out) {
+                        int32_t c = vo[a] + fd.f_out[k][a];   // output tiler (Fig. 6), toroidal
+                        if (c >= fd.s_out[a]) c -= fd.s_out[a];
+                        off += c * int32_t(fd.st_out[a]);
+                    }
+                }
+            }
+            out[off] = tile;
+        }
+    }
+}
+
+// (mul, sh) with floor(x / d) == (umulhi(x, mul) + x) >> sh for every 0 <= x <= 2^31 (1 <= d <= 2^31):
+// sh = ceil(log2 d), mul = floor(2^32 (2^sh - d) / d) + 1 (the round-up method; the 33-bit sum
+// umulhi + x stays below 2^32 because x <= 2^31).  Checked exhaustively for small d in tests/test_abi.py.
+void magic_u31(uint32_t d, uint32_t* mul, uint32_t* sh) {
+    uint32_t s = 0;
+    while (s < 32 && (uint64_t(1) << s) < uint64_t(d)) ++s;
+    *sh = s;
+    *mul = uint32_t(((uint64_t(1) << 32) * ((uint64_t(1) << s) - uint64_t(d))) / uint64_t(d) + 1);
+}
+
+// AOL_FILTER_LEGACY=1 selects the per-window-load kernels (A/B measurements only).
+bool getenv_flag_filter_legacy() {
+    static const bool v = [] {
+        const char* e = std::getenv("AOL_FILTER_LEGACY");
+        return e && e[0] == '1';
+    }();
+    return v;
+}
+
 int64_t emod(int64_t a, int64_t m) {
     const int64_t r = a % m;
     return r < 0 ? r + m : r;
@@ -384,6 +537,11 @@ aol_status_t aol_filter_apply(const aol_filter_t* f, const int32_t* d_in, int32_
     }
     fill_side(&f->in, fd.s_in, fd.st_in, fd.o_in, fd.P_in);
     fill_side(&f->out, fd.s_out, fd.st_out, fd.o_out, fd.P_out);
+    for (int a = 0; a < AOL_MAX_RANK; ++a) {
+        if (a < fd.ra_in) magic_u31(uint32_t(fd.s_in[a]), &fd.mi_mul[a], &fd.mi_sh[a]);
+        if (a < fd.ra_out) magic_u31(uint32_t(fd.s_out[a]), &fd.mo_mul[a], &fd.mo_sh[a]);
+    }
+    magic_u31(uint32_t(f->divisor < 0 ? -int64_t(f->divisor) : int64_t(f->divisor)), &fd.dv_mul, &fd.dv_sh);
     for (int k = 0; k < fd.n_win; ++k) fd.start[k] = f->window_start[k];
     fill_offsets(&f->in, fd.n_in, fd.f_in);
     fill_offsets(&f->out, fd.n_win, fd.f_out);
@@ -410,6 +568,29 @@ aol_status_t aol_filter_apply(const aol_filter_t* f, const int32_t* d_in, int32_
             for (int j = 0; j < t->rep_rank; ++j) bound += __int128(t->array_shape[a]) * t->rep_shape[j];
             if (bound >= (__int128(1) << 31)) small = false;
         }
+    if (small && fd.n_in <= 16 && !(getenv_flag_filter_legacy())) {
+        // pattern contiguous in the array (element p at base + p): 128-bit loads; the padded tail of the last
+        // vector is read only when it stays inside the input array (checked per repetition in the kernel)
+        int32_t contig = (reinterpret_cast<uintptr_t>(d_in) % 16) == 0;
+        for (int p = 0; p < fd.n_in; ++p) contig &= fd.lin_in[p] == p;
+        const int32_t in_elems = int32_t(elems(f->in.array_shape, f->in.array_rank));
+        const int np = (fd.n_in + 3) / 4 * 4;
+        auto go = [&](auto kd) {
+            constexpr int DD = decltype(kd)::value;
+            switch (np) {
+                case 4: filter32_reg_kernel<DD, 4><<<grid, 256, 0, s>>>(fd, d_in, d_out, in_elems, contig); break;
+                case 8: filter32_reg_kernel<DD, 8><<<grid, 256, 0, s>>>(fd, d_in, d_out, in_elems, contig); break;
+                case 12: filter32_reg_kernel<DD, 12><<<grid, 256, 0, s>>>(fd, d_in, d_out, in_elems, contig); break;
+                default: filter32_reg_kernel<DD, 16><<<grid, 256, 0, s>>>(fd, d_in, d_out, in_elems, contig); break;
+            }
+        };
+        if (D <= 2) go(std::integral_constant<int, 2>{});
+        else if (D <= 3) go(std::integral_constant<int, 3>{});
+        else if (D <= 4) go(std::integral_constant<int, 4>{});
+        else go(std::integral_constant<int, 8>{});
+        AOL_LAUNCH_CHECK("filter32_reg_kernel");
+        return AOL_OK;
+    }
     if (small) {
         if (D <= 2) filter32_kernel<2><<<grid, 256, 0, s>>>(fd, d_in, d_out);
         else if (D <= 3) filter32_kernel<3><<<grid, 256, 0, s>>>(fd, d_in, d_out);

@@ -212,6 +212,27 @@ def test_kernel_division_identities():
     assert np.array_equal((p >> 18) + (T < 0), np.trunc(T / 6).astype(np.int64))
 
 
+def test_magic_division_formula():
+    """filter.cu's magic_u31: floor(x/d) == (umulhi(x, mul) + x) >> sh for 0 <= x <= 2^31, with
+    sh = ceil(log2 d), mul = floor(2^32 (2^sh - d) / d) + 1 (also the repetition decomposition's formula).
+    Exhaustive over x < 2^16 for d < 300, and the extremes / random x for large d."""
+    def magic(d):
+        sh = 0
+        while (1 << sh) < d:
+            sh += 1
+        return ((1 << 32) * ((1 << sh) - d)) // d + 1, sh
+
+    rng = np.random.default_rng(5)
+    xs_small = np.arange(0, 1 << 16, dtype=np.uint64)
+    for d in list(range(1, 300)) + [1000, 1080, 1920, 12345, 65537, (1 << 30) + 3, (1 << 31) - 1, 1 << 31]:
+        mul, sh = magic(d)
+        xs = xs_small if d < 300 else np.concatenate(
+            [rng.integers(0, (1 << 31) + 1, 200000, dtype=np.uint64), np.array([0, d - 1, d, (1 << 31) - 1, 1 << 31],
+                                                                             dtype=np.uint64)])
+        q = (((xs * np.uint64(mul)) >> np.uint64(32)) + xs) >> np.uint64(sh)
+        assert np.array_equal(q, xs // np.uint64(d)), d
+
+
 def test_c_example_builds_against_header():
     """examples/aol_example.c compiles and links against include/aol.h + libaol.so with gcc (C99)."""
     import subprocess

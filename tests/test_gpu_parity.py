@@ -322,6 +322,54 @@ def test_filter_random_tilers_vs_oracle(orc, seed):
     assert np.array_equal(out.cpu().numpy(), want)
 
 
+def _task_c(G, starts, L, d):
+    """Fig. 5's task generalised (windows at `starts`, length L, divisor d): tmp/d - tmp%d in C semantics."""
+    S = np.stack([G[..., s:s + L].astype(np.int64).sum(-1) for s in starts], -1)
+    q = np.sign(S) * np.sign(d) * (np.abs(S) // abs(d))
+    return (q - (S - q * d)).astype(np.int32)
+
+
+@pytest.mark.parametrize("seed", range(40))
+def test_filter_random_windows_and_divisors(orc, seed):
+    """f3 beyond the paper's two filters: random pattern sizes (1..20: register-pattern kernel up to 16,
+    per-window kernel above), window sets and divisors of both signs.  Expected = oracle gather -> the
+    task written out with C division -> oracle scatter."""
+    rng = np.random.default_rng(1300 + seed)
+    n_in = int(rng.integers(1, 21))
+    L = int(rng.integers(1, n_in + 1))
+    n_out = int(rng.integers(1, 9))
+    starts = [int(rng.integers(0, n_in - L + 1)) for _ in range(n_out)]
+    d = int(rng.choice([1, 2, 3, 5, 6, 7, 9, 100, 12345, -1, -3, -6, -77, (1 << 30) + 3]))
+    contiguous = seed % 2 == 0
+    if contiguous:   # pattern along the unit-stride dim of a wide array (128-bit loads), wrap only at row ends
+        arr_in = [int(rng.integers(1, 4)), int(rng.integers(1, 5)), 8 * int(rng.integers(4, 40))]
+        step = int(rng.integers(1, 9))
+        rep = [arr_in[0], arr_in[1], arr_in[2] // step]
+        o_in, P_in, F_in = [0, 0, int(rng.integers(0, 3))], [[1, 0, 0], [0, 1, 0], [0, 0, step]], [[0], [0], [1]]
+    else:
+        ra = int(rng.integers(1, 4))
+        rep = [int(rng.integers(1, 6)) for _ in range(int(rng.integers(1, 3)))]
+        arr_in = [int(rng.integers(2, 17)) for _ in range(ra)]
+        o_in = [int(rng.integers(-2 * s, 2 * s + 1)) for s in arr_in]
+        P_in = [[int(rng.integers(-4, 10)) for _ in rep] for _ in range(ra)]
+        F_in = [[int(rng.integers(-4, 10))] for _ in range(ra)]
+    nrep = int(np.prod(rep))
+    arr_out = [nrep, n_out]
+    strides = [int(np.prod(rep[j + 1:])) for j in range(len(rep))]
+    P_out, F_out = [strides, [0] * len(rep)], [[0], [1]]
+    xh = np.asarray(rng.integers(-5000, 5000, size=arr_in)).astype(np.int32)
+    oti = orc.make_tiler(arr_in, rep, [n_in], o_in, P_in, F_in)
+    oto = orc.make_tiler(arr_out, rep, [n_out], [0, 0], P_out, F_out)
+    bg = np.full(arr_out, -99, np.int32)
+    want = orc.scatter(oto, _task_c(orc.gather(oti, xh), starts, L, d), bg)
+    f = aol.make_filter(aol.make_tiler(arr_in, rep, [n_in], o_in, P_in, F_in),
+                        aol.make_tiler(arr_out, rep, [n_out], [0, 0], P_out, F_out), starts, L, d)
+    out = torch.from_numpy(bg.copy()).cuda()
+    aol.filter_apply(f, torch.from_numpy(xh).cuda(), out=out)
+    torch.cuda.synchronize()
+    assert np.array_equal(out.cpu().numpy(), want), (n_in, L, starts, d)
+
+
 def test_tiler_paper_presets_on_gpu(orc):
     H, W = 27, 64
     xh = synth.planes(4, 1, H, W)[0]
