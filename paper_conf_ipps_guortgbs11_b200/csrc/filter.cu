@@ -45,6 +45,8 @@ struct FilterDev {
     // magic numbers: x mod s_in/s_out (x < 2^31) and |S| / |divisor| (|S| <= 2^31) as (umulhi(x, mul) + x) >> sh
     uint32_t mi_mul[AOL_MAX_RANK], mi_sh[AOL_MAX_RANK], mo_mul[AOL_MAX_RANK], mo_sh[AOL_MAX_RANK];
     uint32_t dv_mul, dv_sh;
+    // (32 * P[a][last rep dim]) mod s: reference-point step between a lane's consecutive repetitions
+    int32_t st32_in[AOL_MAX_RANK], st32_out[AOL_MAX_RANK];
 };
 
 // floor(x / d) for 0 <= x <= 2^31 and the host-computed (mul, sh) of d (1 <= d < 2^31)
@@ -252,38 +254,70 @@ __global__ void __launch_bounds__(256) filter32_reg_kernel(const FilterDev fd, c
     __syncthreads();
     int32_t* my = pre + threadIdx.x;
     const int32_t nrep = int32_t(fd.nrep);
-    for (int32_t r = int32_t(blockIdx.x * blockDim.x + threadIdx.x); r < nrep; r += int32_t(gridDim.x * blockDim.x)) {
-        int32_t vi[D], vo[D];
+    // Each warp takes chunks of 32 * kT consecutive repetitions; lane l handles l, l + 32, ...  (coalesced
+    // across the warp).  Only a lane's first repetition of a chunk, and one whose innermost repetition index
+    // carries into the next dimension, decomposes its index (magic-number divisions + mod); the others step
+    // the reference points o' + P'.r by 32 columns of P' with one conditional subtract per dimension.
+    constexpr int kT = 8;
+    const int32_t lane = int32_t(threadIdx.x & 31u);
+    const int32_t nchunks = (nrep + 32 * kT - 1) / (32 * kT);
+    const int32_t nwarps = int32_t((gridDim.x * blockDim.x) >> 5);
+    const int32_t ext_last = fd.rr > 0 ? fd.rep_ext[fd.rr - 1] : 1;
+    for (int32_t chunk = int32_t((blockIdx.x * blockDim.x + threadIdx.x) >> 5); chunk < nchunks; chunk += nwarps) {
+    int32_t vi[D], vo[D], ilast = 0;
+    bool have = false;
+    for (int32_t t = 0, r = chunk * 32 * kT + lane; t < kT && r < nrep; ++t, r += 32) {
+        if (have && ilast + 32 < ext_last) {
+            ilast += 32;
 #pragma unroll
-        for (int a = 0; a < D; ++a) {
-            vi[a] = fd.o_in[a];
-            vo[a] = fd.o_out[a];
-        }
-        uint32_t n = uint32_t(r);
-#pragma unroll
-        for (int j = D - 1; j >= 0; --j) {
-            if (j < fd.rr) {
-                const uint32_t q = (__umulhi(n, fd.fd_mul[j]) + n) >> fd.fd_shift[j];
-                const int32_t i = int32_t(n - q * uint32_t(fd.rep_ext[j]));
-                n = q;
-#pragma unroll
-                for (int a = 0; a < D; ++a) {   // reference points o' + P'.r (Section IV)
-                    vi[a] += fd.P_in[a][j] * i;
-                    vo[a] += fd.P_out[a][j] * i;
+            for (int a = 0; a < D; ++a) {
+                if (a < fd.ra_in) {
+                    vi[a] += fd.st32_in[a];
+                    if (vi[a] >= fd.s_in[a]) vi[a] -= fd.s_in[a];
                 }
+                if (a < fd.ra_out) {
+                    vo[a] += fd.st32_out[a];
+                    if (vo[a] >= fd.s_out[a]) vo[a] -= fd.s_out[a];
+                }
+            }
+        } else {
+            have = true;
+#pragma unroll
+            for (int a = 0; a < D; ++a) {
+                vi[a] = fd.o_in[a];
+                vo[a] = fd.o_out[a];
+            }
+            uint32_t n = uint32_t(r);
+#pragma unroll
+            for (int j = D - 1; j >= 0; --j) {
+                if (j < fd.rr) {
+                    const uint32_t q = (__umulhi(n, fd.fd_mul[j]) + n) >> fd.fd_shift[j];
+                    const int32_t i = int32_t(n - q * uint32_t(fd.rep_ext[j]));
+                    n = q;
+                    if (j == fd.rr - 1) ilast = i;
+#pragma unroll
+                    for (int a = 0; a < D; ++a) {   // reference points o' + P'.r (Section IV)
+                        vi[a] += fd.P_in[a][j] * i;
+                        vo[a] += fd.P_out[a][j] * i;
+                    }
+                }
+            }
+#pragma unroll
+            for (int a = 0; a < D; ++a) {   // mod s (all terms >= 0 and < 2^31): magic-number division
+                if (a < fd.ra_in) vi[a] -= int32_t(udiv_magic(uint32_t(vi[a]), fd.mi_mul[a], fd.mi_sh[a])) * fd.s_in[a];
+                if (a < fd.ra_out)
+                    vo[a] -= int32_t(udiv_magic(uint32_t(vo[a]), fd.mo_mul[a], fd.mo_sh[a])) * fd.s_out[a];
             }
         }
         bool in_ok = true, out_ok = true;
         int32_t base_in = 0, base_out = 0;
 #pragma unroll
-        for (int a = 0; a < D; ++a) {   // mod s (all terms >= 0 and < 2^31): magic-number division
+        for (int a = 0; a < D; ++a) {
             if (a < fd.ra_in) {
-                vi[a] -= int32_t(udiv_magic(uint32_t(vi[a]), fd.mi_mul[a], fd.mi_sh[a])) * fd.s_in[a];
                 in_ok &= vi[a] + fd.fmax_in[a] < fd.s_in[a];
                 base_in += vi[a] * int32_t(fd.st_in[a]);
             }
             if (a < fd.ra_out) {
-                vo[a] -= int32_t(udiv_magic(uint32_t(vo[a]), fd.mo_mul[a], fd.mo_sh[a])) * fd.s_out[a];
                 out_ok &= vo[a] + fd.fmax_out[a] < fd.s_out[a];
                 base_out += vo[a] * int32_t(fd.st_out[a]);
             }
@@ -354,6 +388,7 @@ __global__ void __launch_bounds__(256) filter32_reg_kernel(const FilterDev fd, c
             }
             out[off] = tile;
         }
+    }
     }
 }
 
@@ -542,6 +577,10 @@ aol_status_t aol_filter_apply(const aol_filter_t* f, const int32_t* d_in, int32_
         if (a < fd.ra_out) magic_u31(uint32_t(fd.s_out[a]), &fd.mo_mul[a], &fd.mo_sh[a]);
     }
     magic_u31(uint32_t(f->divisor < 0 ? -int64_t(f->divisor) : int64_t(f->divisor)), &fd.dv_mul, &fd.dv_sh);
+    for (int a = 0; a < AOL_MAX_RANK && fd.rr > 0; ++a) {
+        if (a < fd.ra_in) fd.st32_in[a] = int32_t(emod(32 * int64_t(fd.P_in[a][fd.rr - 1]), fd.s_in[a]));
+        if (a < fd.ra_out) fd.st32_out[a] = int32_t(emod(32 * int64_t(fd.P_out[a][fd.rr - 1]), fd.s_out[a]));
+    }
     for (int k = 0; k < fd.n_win; ++k) fd.start[k] = f->window_start[k];
     fill_offsets(&f->in, fd.n_in, fd.f_in);
     fill_offsets(&f->out, fd.n_win, fd.f_out);
