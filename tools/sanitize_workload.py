@@ -26,7 +26,8 @@ def main():
     kernels = [int(k) for k in args.kernels.split(",")]
     torch.cuda.set_device(0)
     ok = True
-    shapes = [(2, 3, 27, 64), (1, 1, 9, 32), (1, 2, 18, 352), (2, 2, 18, 256)]
+    # W = 1040: uint8 two-repetitions-per-thread path with a partly idle warp and 1-D bulk copies
+    shapes = [(2, 3, 27, 64), (1, 1, 9, 32), (1, 2, 18, 352), (2, 2, 18, 256), (1, 1, 18, 1040)]
     if args.widths:
         shapes = [sh for sh in shapes if str(sh[3]) in args.widths.split(",")]
     for (N, C, H, W) in shapes:
@@ -71,6 +72,12 @@ def main():
     G2 = aol.tiler_gather(tw, A[:9, :10].contiguous())
     C2 = torch.zeros((9, 10), dtype=torch.int32, device="cuda")
     aol.tiler_scatter(tw, G2, C2, mode="sequential")
+    # generic run-time filters (register-pattern kernel: 128-bit contiguous path, wrapping path, stepping)
+    P, H, W = 2, 18, 256
+    x = aol.synth_frames(3, 0, 1, P, H, W, "uniform")[0]
+    y = aol.filter_apply(aol.filter_preset(aol.FILTER_H, P, H, W), x)
+    z = aol.filter_apply(aol.filter_preset(aol.FILTER_V, P, H, 3 * W // 8), y)
+    ok &= torch.equal(z, aol.downscale_frame(x.unsqueeze(1))[0][:, 0])
     torch.cuda.synchronize()
     print("sanitize workload:", "OK" if ok else "MISMATCH")
     return 0 if ok else 1
