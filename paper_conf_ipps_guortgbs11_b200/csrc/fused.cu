@@ -51,13 +51,20 @@ bool tma_shape_ok(aol_dtype_t dt, int64_t planes, int64_t channels, int64_t H, i
     if (H < 9 || W / 8 > kMaxConsumers) return false;
     // checksum weights (1 + frame-local output index) are computed in 32 bits
     if (channels * (4 * (H / 9)) * (3 * (W / 8)) >= (int64_t(1) << 32) - 1) return false;
-    if (dt == AOL_I32) return W % 32 == 0 && W / 32 <= 256 && planes * H < (int64_t(1) << 31);
+    // int32: {32, W/32, 3}-element boxes under SWIZZLE_128B, or {8, W/8, 3} under SWIZZLE_32B when W % 32 != 0
+    // (a box dimension holds at most 256 elements)
+    if (dt == AOL_I32)
+        return (W % 32 == 0 ? W / 32 <= 256 : W / 8 <= 256) && planes * H < (int64_t(1) << 31);
     if (dt == AOL_U8) return W % 16 == 0;   // 1-D bulk copies: 16-byte granularity
     return false;
 }
 
-KernelFn pick(aol_dtype_t dt, bool checksum, int kr, int block, int cps) {
-    return dt == AOL_U8 ? tma_kernel_u8(checksum, kr, block, cps) : tma_kernel_i32(checksum, block, cps);
+// int32 frames whose width is not a multiple of 32 use 32-byte lines (SWIZZLE_32B)
+bool swz32_layout(aol_dtype_t dt, int64_t W) { return dt == AOL_I32 && W % 32 != 0; }
+
+KernelFn pick(aol_dtype_t dt, bool checksum, int kr, int64_t W, int block, int cps) {
+    return dt == AOL_U8 ? tma_kernel_u8(checksum, kr, block, cps)
+                        : tma_kernel_i32(checksum, swz32_layout(dt, W), block, cps);
 }
 
 // Shared-memory geometry of the TMA ring: one stage = one row triple.
@@ -88,14 +95,15 @@ aol_status_t encode_row_map(CUtensorMap* map, aol_dtype_t dt, const void* base, 
     aol_status_t st = get_encode_fn(&encode);
     if (st != AOL_OK) return st;
     const bool i32 = dt == AOL_I32;
-    const cuuint64_t inner = i32 ? 32 : 128, es = i32 ? 4 : 1;
+    const bool s32 = swz32_layout(dt, W);
+    const cuuint64_t inner = i32 ? (s32 ? 8 : 32) : 128, es = i32 ? 4 : 1;
     const cuuint64_t gdim[3] = {inner, cuuint64_t(W) / inner, cuuint64_t(rows)};
     const cuuint64_t gstride[2] = {inner * es, cuuint64_t(W) * es};
     const cuuint32_t box[3] = {cuuint32_t(inner), cuuint32_t(W / int64_t(inner)), 3};
     const cuuint32_t estr[3] = {1, 1, 1};
     CUresult cr = encode(map, i32 ? CU_TENSOR_MAP_DATA_TYPE_INT32 : CU_TENSOR_MAP_DATA_TYPE_UINT8, 3,
                          const_cast<void*>(base), gdim, gstride, box, estr, CU_TENSOR_MAP_INTERLEAVE_NONE,
-                         i32 ? CU_TENSOR_MAP_SWIZZLE_128B : CU_TENSOR_MAP_SWIZZLE_NONE,
+                         i32 ? (s32 ? CU_TENSOR_MAP_SWIZZLE_32B : CU_TENSOR_MAP_SWIZZLE_128B) : CU_TENSOR_MAP_SWIZZLE_NONE,
                          CU_TENSOR_MAP_L2_PROMOTION_L2_256B, CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
     if (cr != CUDA_SUCCESS) {
         set_error("cuTensorMapEncodeTiled failed (CUresult %d)", int(cr));
@@ -151,7 +159,8 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, const void* d_in, const int32_t* d
             int occ = 0;
             const int smem = smem_bytes(geom, stages);
             if (stages >= 2 && cps > 1)
-                occ = kernel_occupancy(reinterpret_cast<const void*>(pick(in_dtype, true, kr, block, cps)), block, smem);
+                occ = kernel_occupancy(reinterpret_cast<const void*>(pick(in_dtype, true, kr, W, block, cps)), block,
+                                       smem);
             if (cps == 1) occ = 1;   // one CTA always fits once its shared memory does
             if ((stages >= 2 && occ >= cps) || cps == 1 || o.ctas_per_sm > 0) {
                 if (stages < 2) tma_ok = false;
@@ -161,7 +170,8 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, const void* d_in, const int32_t* d
     }
     if (o.kernel == 1 && !tma_ok) {
         set_error("TMA fused kernel requested but unsupported for this shape/dtype/alignment "
-                  "(int32: W %% 32 == 0 and W <= 7680; uint8: W %% 16 == 0 and W <= 7936; 16-byte aligned buffers)");
+                  "(int32: W <= 7680 when W %% 32 == 0, else W <= 2048; uint8: W %% 16 == 0 and W <= 7936; "
+                  "16-byte aligned buffers)");
         return AOL_E_SHAPE;
     }
     if (o.kernel == 2) tma_ok = false;
@@ -253,7 +263,7 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
     a.Wo = Wo;
     a.channels = int32_t(channels);
     a.reps = int32_t(W / 8);
-    a.segs = int32_t(W / 32);
+    a.segs = int32_t(swz32_layout(in_dtype, W) ? W / 8 : W / 32);   // int32 lines per row
     a.triples_per_plane = int32_t(H / 3);
     a.nbands = int32_t(H / 9);
     a.bands_per_unit = plan.bands_per_unit;
@@ -268,7 +278,7 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
     a.hint_stores = (plan.flags & AOL_FLAG_EVICT_FIRST_STORES) ? 1 : 0;
     a.blocked_units = (plan.flags & AOL_FLAG_BLOCKED_UNITS) ? 1 : 0;
 
-    KernelFn k = pick(in_dtype, d_cs != nullptr, plan.reps_per_thread, plan.block, plan.ctas_per_sm);
+    KernelFn k = pick(in_dtype, d_cs != nullptr, plan.reps_per_thread, W, plan.block, plan.ctas_per_sm);
     aol_status_t st_attr = kernel_smem(reinterpret_cast<const void*>(k), plan.smem);
     if (st_attr != AOL_OK) return st_attr;
     // With checksums: zero them in a one-CTA kernel and launch the fused kernel as its programmatic

@@ -5,12 +5,15 @@ namespace aol {
 namespace fused {
 KernelFn tma_kernel_i32_cs(int block, int cps);
 KernelFn tma_kernel_i32_nocs(int block, int cps);
+KernelFn tma_kernel_i32s_cs(int block, int cps);
+KernelFn tma_kernel_i32s_nocs(int block, int cps);
 KernelFn tma_kernel_u8_cs(int block, int cps);
 KernelFn tma_kernel_u8_nocs(int block, int cps);
 KernelFn tma_kernel_u8r2_cs(int block, int cps);
 KernelFn tma_kernel_u8r2_nocs(int block, int cps);
 
-KernelFn tma_kernel_i32(bool checksum, int block, int cps) {
+KernelFn tma_kernel_i32(bool checksum, bool swz32, int block, int cps) {
+    if (swz32) return checksum ? tma_kernel_i32s_cs(block, cps) : tma_kernel_i32s_nocs(block, cps);
     return checksum ? tma_kernel_i32_cs(block, cps) : tma_kernel_i32_nocs(block, cps);
 }
 KernelFn tma_kernel_u8(bool checksum, int reps_per_thread, int block, int cps) {

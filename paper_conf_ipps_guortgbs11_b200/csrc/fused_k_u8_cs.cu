@@ -1,8 +1,10 @@
-// Explicit instantiations of fused_tma_kernel<uint8_t, kR=1, checksum=true> (split for parallel builds).
+// Explicit instantiations of fused_tma_kernel<uint8_t, kR=1, kSwz=0, checksum=true> (split for parallel builds).
 #include "fused_kernel.cuh"
 
 namespace aol {
 namespace fused {
-KernelFn tma_kernel_u8_cs(int block, int cps) { return pick_tma_kernel<uint8_t, 1, true>(block, cps); }
+KernelFn tma_kernel_u8_cs(int block, int cps) {
+    return pick_tma_kernel<uint8_t, 1, 0, true>(block, cps);
+}
 }  // namespace fused
 }  // namespace aol

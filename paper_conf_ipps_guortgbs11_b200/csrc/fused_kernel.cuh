@@ -89,7 +89,7 @@ struct FusedArgs {
     int32_t H, W, Ho, Wo;
     int32_t channels;
     int32_t reps;               // W/8  repetitions of the H tiler per row
-    int32_t segs;               // int32 path: W/32 128-byte segments per row
+    int32_t segs;               // int32 path: lines per row (W/32 of 128 B, or W/8 of 32 B with SWIZZLE_32B)
     int32_t triples_per_plane;  // H/3
     int32_t nbands;             // H/9
     int32_t bands_per_unit;
@@ -111,6 +111,13 @@ __device__ __forceinline__ uint32_t swz(uint32_t line, uint32_t chunk) {
     return (line << 7) | (((chunk ^ line) & 7u) << 4);
 }
 
+// Same under SWIZZLE_32B for 32-byte lines (int32 frames with W % 32 != 0: one repetition = one line of
+// 8 elements): the 16-byte chunk index (0/1) XOR line bit 2 (address bit 4 ^= bit 7; 1024-aligned stages).
+// Eight consecutive lines then cover all eight 16-byte bank groups for either chunk: conflict-free LDS.128.
+__device__ __forceinline__ uint32_t swz32(uint32_t line, uint32_t chunk) {
+    return (line << 5) | (((chunk ^ (line >> 2)) & 1u) << 4);
+}
+
 // k-th work unit of this CTA: round-robin (concurrently running CTAs stream adjacent units) or, with
 // AOL_FLAG_BLOCKED_UNITS, a contiguous block of units per CTA.  Returns >= nunits when done.
 __device__ __forceinline__ int64_t unit_of(const FusedArgs& a, int64_t k) {
@@ -123,20 +130,26 @@ __device__ __forceinline__ int64_t unit_of(const FusedArgs& a, int64_t k) {
 struct RepGeom {
     uint32_t off0, off1;  // int32: swizzled offsets of the two chunks within a row's lines; uint8: 8r
     uint32_t offn;        // neighbour repetition's first chunk / word
-    uint32_t seg, segn;   // int32: 128-byte segment of the repetition and of its neighbour
+    uint32_t seg, segn;   // int32: 128-byte segment (32-byte line with kSwz == 32) of the repetition / neighbour
     bool fix;             // read the neighbour from smem instead of the shuffle
 };
 
 // H stage of one input row: the three 6-tap window sums of each of the thread's kR repetitions, T() applied:
 // y[3j + k] = T(window k of repetition j).
-template <typename Tin, int kR>
+template <typename Tin, int kR, int kSwz>
 __device__ __forceinline__ void h_row(uint32_t row_base, uint32_t rr, const RepGeom& g, uint32_t segs, uint32_t W,
                                       int32_t (&y)[3 * kR]) {
     if constexpr (std::is_same<Tin, int32_t>::value) {
         static_assert(kR == 1, "int32 path: one repetition per thread");
         const uint32_t line = rr * segs + g.seg;
-        const int4 q0 = ptx::lds128(row_base + swz(line, g.off0));
-        const int4 q1 = ptx::lds128(row_base + swz(line, g.off1));
+        int4 q0, q1;
+        if constexpr (kSwz == 32) {
+            q0 = ptx::lds128(row_base + swz32(line, 0));
+            q1 = ptx::lds128(row_base + swz32(line, 1));
+        } else {
+            q0 = ptx::lds128(row_base + swz(line, g.off0));
+            q1 = ptx::lds128(row_base + swz(line, g.off1));
+        }
         const int32_t e = q0.x + q0.y;
         const int32_t d = e + q0.z;                 // cols 8r..8r+2: the left neighbour's overlap
         const int32_t q = q0.z + q0.w;
@@ -145,7 +158,10 @@ __device__ __forceinline__ void h_row(uint32_t row_base, uint32_t rr, const RepG
         const int32_t qp = q + p;
         int32_t dn = __shfl_down_sync(0xffffffffu, d, 1);
         int4 qn = q0;   // lane 31 / wrapping repetition: neighbour chunk from smem (predicated, no branch)
-        ptx::lds128_if(qn, row_base + swz(rr * segs + g.segn, g.offn), g.fix);
+        if constexpr (kSwz == 32)
+            ptx::lds128_if(qn, row_base + swz32(rr * segs + g.segn, 0), g.fix);
+        else
+            ptx::lds128_if(qn, row_base + swz(rr * segs + g.segn, g.offn), g.fix);
         dn = g.fix ? qn.x + qn.y + qn.z : dn;
         y[0] = task_T(e + qp);            // window cols 0..5
         y[1] = task_T(qp + f);            // window cols 2..7
@@ -185,7 +201,9 @@ __device__ __forceinline__ void h_row(uint32_t row_base, uint32_t rr, const RepG
 // kR = repetitions of the H tiler per consumer thread: 1 for int32 (two LDS.128 already cover one repetition's
 // 8 columns); 1 or 2 for uint8 input, whose 16 bytes for two repetitions come in one LDS.128 and whose per-stage
 // bookkeeping (mbarrier wait/arrive, addressing) two repetitions then share (the host picks, fused.cu).
-template <typename Tin, int kR, bool kChecksum, int kMaxThreads, int kMinBlocks>
+// kSwz = the int32 smem layout: 128 (SWIZZLE_128B, W % 32 == 0) or 32 (SWIZZLE_32B, other W % 8 == 0);
+// unused (0) for uint8.
+template <typename Tin, int kR, int kSwz, bool kChecksum, int kMaxThreads, int kMinBlocks>
 __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
     fused_tma_kernel(const __grid_constant__ CUtensorMap tmap, const FusedArgs a) {
     constexpr bool kI32 = std::is_same<Tin, int32_t>::value;
@@ -258,7 +276,11 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
     const int rn = (r + kR == a.reps) ? 0 : r + kR;  // next thread's repetition (toroidal, Fig. 11 '% 1920')
     RepGeom g;
     g.fix = (lane == 31) || (r + 1 == a.reps);
-    if constexpr (kI32) {
+    if constexpr (kI32 && kSwz == 32) {
+        g.seg = uint32_t(r);   // one 32-byte line per repetition
+        g.segn = uint32_t(rn);
+        g.off0 = g.off1 = g.offn = 0;
+    } else if constexpr (kI32) {
         g.seg = uint32_t(r) >> 2;
         g.segn = uint32_t(rn) >> 2;
         g.off0 = (uint32_t(r) & 3u) << 1;   // chunk indices within the 128-byte line
@@ -362,7 +384,7 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
 #pragma unroll
                 for (int m = 0; m < kC; ++m) y[rr][m] = int32_t(sb) + rr;
 #else
-                h_row<Tin, kR>(sb, uint32_t(rr), g, segs, Wu, y[rr]);
+                h_row<Tin, kR, kSwz>(sb, uint32_t(rr), g, segs, Wu, y[rr]);
 #endif
             }
             __syncwarp();
@@ -519,23 +541,23 @@ __global__ void __launch_bounds__(256)
 using KernelFn = void (*)(const CUtensorMap, const FusedArgs);
 
 // Explicit instantiations live in fused_k_*.cu (compiled in parallel); these pick one.
-KernelFn tma_kernel_i32(bool checksum, int block, int cps);
+KernelFn tma_kernel_i32(bool checksum, bool swz32, int block, int cps);
 KernelFn tma_kernel_u8(bool checksum, int reps_per_thread, int block, int cps);
 
-template <typename Tin, int kR, bool kChecksum>
+template <typename Tin, int kR, int kSwz, bool kChecksum>
 KernelFn pick_tma_kernel(int block, int cps) {
     if constexpr (kR == 2) {
         // two repetitions per thread take ~126 registers: bounds that never force spills below 1024 threads
-        if (block <= 160 && cps >= 3) return fused_tma_kernel<Tin, kR, kChecksum, 160, 3>;
-        if (block <= 256 && cps >= 2) return fused_tma_kernel<Tin, kR, kChecksum, 256, 2>;
-        if (block <= 512) return fused_tma_kernel<Tin, kR, kChecksum, 512, 1>;
-        return fused_tma_kernel<Tin, kR, kChecksum, 1024, 1>;
+        if (block <= 160 && cps >= 3) return fused_tma_kernel<Tin, kR, kSwz, kChecksum, 160, 3>;
+        if (block <= 256 && cps >= 2) return fused_tma_kernel<Tin, kR, kSwz, kChecksum, 256, 2>;
+        if (block <= 512) return fused_tma_kernel<Tin, kR, kSwz, kChecksum, 512, 1>;
+        return fused_tma_kernel<Tin, kR, kSwz, kChecksum, 1024, 1>;
     } else {
-        if (block <= 128 && cps >= 3) return fused_tma_kernel<Tin, kR, kChecksum, 128, 4>;
-        if (block <= 320 && cps >= 3) return fused_tma_kernel<Tin, kR, kChecksum, 320, 3>;
-        if (block <= 320 && cps >= 2) return fused_tma_kernel<Tin, kR, kChecksum, 320, 2>;
-        if (block <= 512) return fused_tma_kernel<Tin, kR, kChecksum, 512, 1>;
-        return fused_tma_kernel<Tin, kR, kChecksum, 1024, 1>;
+        if (block <= 128 && cps >= 3) return fused_tma_kernel<Tin, kR, kSwz, kChecksum, 128, 4>;
+        if (block <= 320 && cps >= 3) return fused_tma_kernel<Tin, kR, kSwz, kChecksum, 320, 3>;
+        if (block <= 320 && cps >= 2) return fused_tma_kernel<Tin, kR, kSwz, kChecksum, 320, 2>;
+        if (block <= 512) return fused_tma_kernel<Tin, kR, kSwz, kChecksum, 512, 1>;
+        return fused_tma_kernel<Tin, kR, kSwz, kChecksum, 1024, 1>;
     }
 }
 

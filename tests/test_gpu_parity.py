@@ -97,9 +97,27 @@ def test_fused_launch_options(orc, opts):
     assert np.array_equal(np_u64(cs), cso)
 
 
-@pytest.mark.parametrize("shape", [(1, 1, 9, 8), (2, 3, 18, 40), (1, 3, 36, 1000)])
+@pytest.mark.parametrize("shape", [(1, 1, 9, 8), (2, 3, 18, 40), (1, 3, 36, 1000), (2, 3, 27, 720), (1, 2, 18, 2040)])
+def test_swizzle32_shapes(orc, shape):
+    """int32, W % 32 != 0 (e.g. 720-wide SD frames): the TMA kernel with 32-byte lines under SWIZZLE_32B
+    ({8, W/8, 3} boxes, W <= 2048), against the oracle and the generic kernel, with and without checksums."""
+    N, C, H, W = shape
+    xh = synth.frames(5, 0, N, C, H, W, "signed")
+    zo, cso = run_oracle(orc, xh)
+    assert aol.downscale_frame_plan(N, C, H, W)["kernel"] == 1
+    x = torch.from_numpy(xh).cuda()
+    for opts in (None, {"kernel": 1, "ctas_per_sm": 2, "bands_per_unit": 1}, {"kernel": 2}):
+        z, cs = aol.downscale_frame(x, checksums=True, opts=opts)
+        z2, _ = aol.downscale_frame(x, opts=opts)
+        torch.cuda.synchronize()
+        assert np.array_equal(z.cpu().numpy(), zo), opts
+        assert np.array_equal(z2.cpu().numpy(), zo), opts
+        assert np.array_equal(np_u64(cs), cso), opts
+
+
+@pytest.mark.parametrize("shape", [(1, 1, 9, 2056), (1, 2, 18, 4008)])
 def test_generic_only_shapes(orc, shape):
-    """W % 32 != 0: the planner must pick the generic fused kernel."""
+    """int32, W % 32 != 0 and W > 2048 (a box dimension holds <= 256 lines): the generic fused kernel."""
     N, C, H, W = shape
     xh = synth.frames(5, 0, N, C, H, W, "signed")
     zo, cso = run_oracle(orc, xh)
