@@ -85,16 +85,19 @@ def measured_peak():
 
 
 def ncu_traffic(a):
-    """Per-launch DRAM bytes from the committed `ncu --set full` summary, if it matches this workload."""
+    """(per-launch DRAM bytes, ncu DRAM utilisation in % of peak, capture tag) from the committed
+    `ncu --set full` summary, if it matches this workload; else (None, None, None)."""
     path = os.path.join(ROOT, "profiles", "ncu_traffic.json")
     try:
         with open(path) as f:
             d = json.load(f)
         key = f"{a.frames}x{a.channels}x{a.H}x{a.W}:{a.dtype}"
         e = d.get(key)
-        return None if e is None else float(e["dram_bytes_per_launch"])
+        if e is None:
+            return None, None, None
+        return float(e["dram_bytes_per_launch"]), e.get("dram_pct_of_peak"), e.get("tag")
     except Exception:
-        return None
+        return None, None, None
 
 
 class ClockSampler:
@@ -351,7 +354,7 @@ def main():
     # algorithmic bytes over kernel time, summed over this rank's launches (all equal in the default mode)
     achieved = bpf * sum(launch_frames) / (sum(launch_ms) / 1000.0) / 1e9
     peak, peak_src = measured_peak()
-    traffic = ncu_traffic(a)
+    traffic, dram_pct, ncu_tag = ncu_traffic(a)
     line = {
         "metric": METRIC, "value": value, "unit": "frames/s", "n_gpus": world, "steps": a.steps,
         "warmup": a.warmup, "ms_per_step": max_ms / a.steps, "higher_is_better": True,
@@ -365,6 +368,9 @@ def main():
                    "plan": plan},
         "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s", "frac": achieved / peak,
                      "traffic": traffic, "peak_source": peak_src,
+                     # the copy peak is half writes while this path is ~86 % reads, so frac can exceed 1; ncu's
+                     # DRAM utilisation of the same launch (committed capture) is the direct measure
+                     "ncu_dram_pct_of_peak": dram_pct, "ncu_capture": ncu_tag,
                      "algorithmic_bytes_per_launch": bpf * calls[0],
                      "avg_launch_ms": avg_launch_s * 1000.0, "min_launch_ms": min(launch_ms)},
         # per call: zero_checksums_kernel + the fused kernel (its programmatic dependent)

@@ -62,7 +62,8 @@ def main():
         path = os.path.join(prof_dir, "ncu_traffic.json")
         allv = json.load(open(path)) if os.path.exists(path) else {}
         allv[key] = {"dram_bytes_per_launch": rb + wb, "dram_read": rb, "dram_write": wb, "tag": tag,
-                     "duration": d["gpu__time_duration.sum"][0] + " " + d["gpu__time_duration.sum"][1]}
+                     "duration": d["gpu__time_duration.sum"][0] + " " + d["gpu__time_duration.sum"][1],
+                     "dram_pct_of_peak": float(d["gpu__dram_throughput.avg.pct_of_peak_sustained_elapsed"][0])}
         json.dump(allv, open(path, "w"), indent=1)
     # launch list
     with open(launches) as f:
