@@ -213,6 +213,21 @@ AOL_API aol_status_t aol_downscale_frame_ex(const void* d_in, aol_dtype_t in_dty
 AOL_API aol_status_t aol_downscale_frame_plan(aol_dtype_t in_dtype, int64_t frames, int64_t channels, int64_t H,
                                       int64_t W, const aol_launch_opts_t* opts, aol_plan_t* out);
 
+/* The fused downscaler with the output element type chosen (NEXT row f1): out_dtype AOL_I32 (as
+ * aol_downscale_frame_ex) or AOL_I16 -- only with in_dtype AOL_U8, whose outputs lie in [-5, 255]
+ * (P:L260, 8-bit samples): d_out int16 [frames][channels][4H/9][3W/8], 2 bytes per output instead of 4.
+ * The checksums are those of the same integer outputs (identical for both output types).  AOL_E_DTYPE
+ * for other combinations; otherwise as aol_downscale_frame_ex. */
+AOL_API aol_status_t aol_downscale_frame_out(const void* d_in, aol_dtype_t in_dtype, void* d_out,
+                                             aol_dtype_t out_dtype, int64_t frames, int64_t channels, int64_t H,
+                                             int64_t W, uint64_t* d_frame_checksums, const aol_launch_opts_t* opts,
+                                             cudaStream_t s);
+
+/* Report the launch aol_downscale_frame_out would make on the current device. */
+AOL_API aol_status_t aol_downscale_frame_plan_out(aol_dtype_t in_dtype, aol_dtype_t out_dtype, int64_t frames,
+                                                  int64_t channels, int64_t H, int64_t W,
+                                                  const aol_launch_opts_t* opts, aol_plan_t* out);
+
 /* Per-frame checksum of an existing output batch (for the unfused paths):
  * d_out int32 [frames][channels][Ho][Wo] -> d_checksums u64 [frames] (overwritten). */
 AOL_API aol_status_t aol_frame_checksum(const int32_t* d_out, int64_t frames, int64_t channels, int64_t Ho, int64_t Wo,

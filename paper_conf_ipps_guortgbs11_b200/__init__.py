@@ -222,8 +222,9 @@ def _opts(opts) -> Optional[aol_launch_opts_t]:
 
 
 def downscale_frame(x: torch.Tensor, out: Optional[torch.Tensor] = None, checksums=None, opts=None,
-                    stream: Optional[torch.cuda.Stream] = None):
-    """Fused downscaler: x [frames][channels][H][W] (int32 or uint8) -> int32 [frames][channels][4H/9][3W/8].
+                    stream: Optional[torch.cuda.Stream] = None, out_dtype: Optional[torch.dtype] = None):
+    """Fused downscaler: x [frames][channels][H][W] (int32 or uint8) -> [frames][channels][4H/9][3W/8]
+    int32, or int16 (out_dtype=torch.int16, uint8 input only: outputs lie in [-5, 255]).
 
     checksums: None (skip), True (allocate), or a uint64/int64 CUDA tensor [frames].
     Returns (out, checksums_or_None)."""
@@ -232,23 +233,27 @@ def downscale_frame(x: torch.Tensor, out: Optional[torch.Tensor] = None, checksu
     if x.dtype not in (torch.int32, torch.uint8):
         raise TypeError("x must be int32 or uint8")
     N, C, H, W = x.shape
+    odt = out.dtype if out is not None else (out_dtype or torch.int32)
+    if odt not in (torch.int32, torch.int16):
+        raise TypeError("output must be int32 or int16")
     if out is None:
-        out = torch.empty((N, C, 4 * (H // 9), 3 * (W // 8)), dtype=torch.int32, device=x.device)
+        out = torch.empty((N, C, 4 * (H // 9), 3 * (W // 8)), dtype=odt, device=x.device)
     cs = checksums
     if cs is True:
         cs = torch.empty(N, dtype=torch.uint64, device=x.device)
     cs_ptr = _dev(cs, "checksums") if cs is not None else ctypes.c_void_p(0)
     o = _opts(opts)
-    check(lib().aol_downscale_frame_ex(_dev(x, "x"), _TYPED[x.dtype], _dev(out, "out"), N, C, H, W, cs_ptr,
-                                       ctypes.byref(o) if o is not None else None, _stream(stream)))
+    check(lib().aol_downscale_frame_out(_dev(x, "x"), _TYPED[x.dtype], _dev(out, "out"), _TYPED[odt], N, C, H, W,
+                                        cs_ptr, ctypes.byref(o) if o is not None else None, _stream(stream)))
     return out, cs
 
 
-def downscale_frame_plan(frames: int, channels: int, H: int, W: int, dtype=torch.int32, opts=None) -> dict:
+def downscale_frame_plan(frames: int, channels: int, H: int, W: int, dtype=torch.int32, opts=None,
+                         out_dtype=torch.int32) -> dict:
     p = aol_plan_t()
     o = _opts(opts)
-    check(lib().aol_downscale_frame_plan(_TYPED[dtype], frames, channels, H, W,
-                                         ctypes.byref(o) if o is not None else None, ctypes.byref(p)))
+    check(lib().aol_downscale_frame_plan_out(_TYPED[dtype], _TYPED[out_dtype], frames, channels, H, W,
+                                             ctypes.byref(o) if o is not None else None, ctypes.byref(p)))
     return {f: getattr(p, f) for f, _ in aol_plan_t._fields_}
 
 

@@ -92,6 +92,10 @@ SIGNATURES = {
                                 ctypes.POINTER(aol_launch_opts_t), _P], _ST),
     "aol_downscale_frame_plan": ([ctypes.c_int, _I64, _I64, _I64, _I64, ctypes.POINTER(aol_launch_opts_t),
                                   ctypes.POINTER(aol_plan_t)], _ST),
+    "aol_downscale_frame_out": ([_P, ctypes.c_int, _P, ctypes.c_int, _I64, _I64, _I64, _I64, _P,
+                                 ctypes.POINTER(aol_launch_opts_t), _P], _ST),
+    "aol_downscale_frame_plan_out": ([ctypes.c_int, ctypes.c_int, _I64, _I64, _I64, _I64,
+                                      ctypes.POINTER(aol_launch_opts_t), ctypes.POINTER(aol_plan_t)], _ST),
     "aol_frame_checksum": ([_P, _I64, _I64, _I64, _I64, _P, _P], _ST),
     "aol_downscale_frame_host_workspace_bytes": ([ctypes.c_int, _I64, _I64, _I64, _I64], ctypes.c_size_t),
     "aol_downscale_frame_host": ([_P, ctypes.c_int, _P, _I64, _I64, _I64, _I64, _P, _I64, _P, ctypes.c_size_t,

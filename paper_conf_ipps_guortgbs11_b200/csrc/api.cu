@@ -251,11 +251,14 @@ using namespace aol;
 
 namespace {
 
-aol_status_t check_frame_args(const void* d_in, aol_dtype_t in_dtype, const int32_t* d_out, int64_t frames,
-                              int64_t channels, int64_t H, int64_t W) {
+aol_status_t check_frame_args(const void* d_in, aol_dtype_t in_dtype, const void* d_out, int64_t frames,
+                              int64_t channels, int64_t H, int64_t W, aol_dtype_t out_dtype = AOL_I32) {
     if (frames < 0 || channels <= 0 || H <= 0 || W <= 0)
         return fail(AOL_E_INVALID, "frames must be >= 0 and channels, H, W > 0");
     if (in_dtype != AOL_I32 && in_dtype != AOL_U8) return fail(AOL_E_DTYPE, "in_dtype must be AOL_I32 or AOL_U8");
+    if (out_dtype != AOL_I32 && out_dtype != AOL_I16) return fail(AOL_E_DTYPE, "out_dtype must be AOL_I32 or AOL_I16");
+    if (out_dtype == AOL_I16 && in_dtype != AOL_U8)
+        return fail(AOL_E_DTYPE, "AOL_I16 output needs AOL_U8 input (8-bit samples give outputs in [-5, 255])");
     if (W % 8) return fail(AOL_E_SHAPE, "W must be a multiple of 8 (H tiler paving step, Fig. 10)");
     if (H % 9) return fail(AOL_E_SHAPE, "H must be a multiple of 9 (V tiler paving step, reading Z1)");
     const __int128 in_elems = __int128(frames) * channels * H * W;
@@ -266,16 +269,17 @@ aol_status_t check_frame_args(const void* d_in, aol_dtype_t in_dtype, const int3
     return AOL_OK;
 }
 
-aol_status_t frame_ex(const void* d_in, aol_dtype_t in_dtype, int32_t* d_out, int64_t frames, int64_t channels,
-                      int64_t H, int64_t W, uint64_t* d_cs, const aol_launch_opts_t* opts, cudaStream_t s) {
-    aol_status_t st = check_frame_args(d_in, in_dtype, d_out, frames, channels, H, W);
+aol_status_t frame_ex(const void* d_in, aol_dtype_t in_dtype, void* d_out, aol_dtype_t out_dtype, int64_t frames,
+                      int64_t channels, int64_t H, int64_t W, uint64_t* d_cs, const aol_launch_opts_t* opts,
+                      cudaStream_t s) {
+    aol_status_t st = check_frame_args(d_in, in_dtype, d_out, frames, channels, H, W, out_dtype);
     if (st != AOL_OK) return st;
     if (frames == 0) return AOL_OK;
     if (opts && (opts->ctas_per_sm < 0 || opts->ctas_per_sm > 8 || opts->stages < 0 || opts->bands_per_unit < 0 ||
                  opts->kernel < 0 || opts->kernel > 2))
         return fail(AOL_E_INVALID, "launch options out of range");
     FusedPlan plan;
-    st = plan_fused(in_dtype, d_in, d_out, frames, channels, H, W, opts, &plan);
+    st = plan_fused(in_dtype, out_dtype, d_in, d_out, frames, channels, H, W, opts, &plan);
     if (st != AOL_OK) return st;
     return launch_fused(plan, d_in, in_dtype, d_out, frames, channels, H, W, d_cs, s);
 }
@@ -434,23 +438,30 @@ aol_status_t aol_downscale_v(const int32_t* d_in, int32_t* d_out, int64_t planes
 aol_status_t aol_downscale_frame(const void* d_in, aol_dtype_t in_dtype, int32_t* d_out, int64_t frames,
                                  int64_t channels, int64_t H, int64_t W, uint64_t* d_frame_checksums,
                                  cudaStream_t s) {
-    return frame_ex(d_in, in_dtype, d_out, frames, channels, H, W, d_frame_checksums, nullptr, s);
+    return frame_ex(d_in, in_dtype, d_out, AOL_I32, frames, channels, H, W, d_frame_checksums, nullptr, s);
 }
 
 aol_status_t aol_downscale_frame_ex(const void* d_in, aol_dtype_t in_dtype, int32_t* d_out, int64_t frames,
                                     int64_t channels, int64_t H, int64_t W, uint64_t* d_frame_checksums,
                                     const aol_launch_opts_t* opts, cudaStream_t s) {
-    return frame_ex(d_in, in_dtype, d_out, frames, channels, H, W, d_frame_checksums, opts, s);
+    return frame_ex(d_in, in_dtype, d_out, AOL_I32, frames, channels, H, W, d_frame_checksums, opts, s);
 }
 
-aol_status_t aol_downscale_frame_plan(aol_dtype_t in_dtype, int64_t frames, int64_t channels, int64_t H,
-                                      int64_t W, const aol_launch_opts_t* opts, aol_plan_t* out) {
+aol_status_t aol_downscale_frame_out(const void* d_in, aol_dtype_t in_dtype, void* d_out, aol_dtype_t out_dtype,
+                                     int64_t frames, int64_t channels, int64_t H, int64_t W,
+                                     uint64_t* d_frame_checksums, const aol_launch_opts_t* opts, cudaStream_t s) {
+    return frame_ex(d_in, in_dtype, d_out, out_dtype, frames, channels, H, W, d_frame_checksums, opts, s);
+}
+
+aol_status_t aol_downscale_frame_plan_out(aol_dtype_t in_dtype, aol_dtype_t out_dtype, int64_t frames,
+                                          int64_t channels, int64_t H, int64_t W, const aol_launch_opts_t* opts,
+                                          aol_plan_t* out) {
     if (!out) return fail(AOL_E_INVALID, "out is NULL");
-    aol_status_t st = check_frame_args(nullptr, in_dtype, nullptr, 0, channels, H, W);
+    aol_status_t st = check_frame_args(nullptr, in_dtype, nullptr, 0, channels, H, W, out_dtype);
     if (st != AOL_OK) return st;
     if (frames <= 0) return fail(AOL_E_INVALID, "frames must be > 0 to plan");
     FusedPlan p;
-    st = plan_fused(in_dtype, nullptr, nullptr, frames, channels, H, W, opts, &p);
+    st = plan_fused(in_dtype, out_dtype, nullptr, nullptr, frames, channels, H, W, opts, &p);
     if (st != AOL_OK) return st;
     out->kernel = p.kernel;
     out->grid = p.grid;
@@ -462,6 +473,11 @@ aol_status_t aol_downscale_frame_plan(aol_dtype_t in_dtype, int64_t frames, int6
     out->ctas_per_sm = p.ctas_per_sm;
     out->num_sms = p.num_sms;
     return AOL_OK;
+}
+
+aol_status_t aol_downscale_frame_plan(aol_dtype_t in_dtype, int64_t frames, int64_t channels, int64_t H,
+                                      int64_t W, const aol_launch_opts_t* opts, aol_plan_t* out) {
+    return aol_downscale_frame_plan_out(in_dtype, AOL_I32, frames, channels, H, W, opts, out);
 }
 
 aol_status_t aol_frame_checksum(const int32_t* d_out, int64_t frames, int64_t channels, int64_t Ho, int64_t Wo,
@@ -509,7 +525,7 @@ aol_status_t aol_downscale_frame_host(const void* h_in, aol_dtype_t in_dtype, in
                          reinterpret_cast<uint64_t*>(ws + 2 * in_b + 2 * out_b + cs_b)};
 
     FusedPlan plan;
-    st = plan_fused(in_dtype, d_in[0], d_out[0], chunk_frames, channels, H, W, nullptr, &plan);
+    st = plan_fused(in_dtype, AOL_I32, d_in[0], d_out[0], chunk_frames, channels, H, W, nullptr, &plan);
     if (st != AOL_OK) return st;
 
     cudaEvent_t ev_in[2], ev_comp[2], ev_out[2];

@@ -58,12 +58,14 @@ struct FusedPlan {
     int kernel;  // 1 = TMA fused, 2 = generic fused
     int grid, block, smem, stages, bands_per_unit, ctas_per_sm, num_sms, units_per_plane, flags;
     int reps_per_thread;  // kernel 1: H-tiler repetitions per consumer thread (1, or 2 for wide uint8 frames)
+    int out_es;           // output element bytes: 4 (int32) or 2 (int16, uint8 input only)
     int64_t units;
 };
 
-aol_status_t plan_fused(aol_dtype_t in_dtype, const void* d_in, const int32_t* d_out, int64_t frames,
-                        int64_t channels, int64_t H, int64_t W, const aol_launch_opts_t* opts, FusedPlan* plan);
-aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t in_dtype, int32_t* d_out,
+aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void* d_in, const void* d_out,
+                        int64_t frames, int64_t channels, int64_t H, int64_t W, const aol_launch_opts_t* opts,
+                        FusedPlan* plan);
+aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t in_dtype, void* d_out,
                           int64_t frames, int64_t channels, int64_t H, int64_t W, uint64_t* d_cs, cudaStream_t s);
 
 aol_status_t launch_downscale_h(const int32_t* d_in, int32_t* d_out, int64_t planes, int64_t H, int64_t W,

@@ -62,8 +62,8 @@ bool tma_shape_ok(aol_dtype_t dt, int64_t planes, int64_t channels, int64_t H, i
 // int32 frames whose width is not a multiple of 32 use 32-byte lines (SWIZZLE_32B)
 bool swz32_layout(aol_dtype_t dt, int64_t W) { return dt == AOL_I32 && W % 32 != 0; }
 
-KernelFn pick(aol_dtype_t dt, bool checksum, int kr, int64_t W, int block, int cps) {
-    return dt == AOL_U8 ? tma_kernel_u8(checksum, kr, block, cps)
+KernelFn pick(aol_dtype_t dt, int out_es, bool checksum, int kr, int64_t W, int block, int cps) {
+    return dt == AOL_U8 ? tma_kernel_u8(checksum, out_es == 2, kr, block, cps)
                         : tma_kernel_i32(checksum, swz32_layout(dt, W), block, cps);
 }
 
@@ -71,15 +71,15 @@ KernelFn pick(aol_dtype_t dt, bool checksum, int kr, int64_t W, int block, int c
 struct RingGeom {
     uint32_t stage_bytes;   // 3 rows of the input
     uint32_t stage_stride;  // rounded up: 1024 B (SWIZZLE_128B atom) for int32, 128 B for uint8
-    uint32_t out_bytes;     // one band of output: 4 rows of Wo int32
+    uint32_t out_bytes;     // one band of output: 4 rows of Wo output elements
 };
 
-RingGeom ring_geom(aol_dtype_t dt, int64_t W) {
+RingGeom ring_geom(aol_dtype_t dt, int out_es, int64_t W) {
     const uint32_t es = dt == AOL_U8 ? 1u : 4u, align = dt == AOL_U8 ? 128u : 1024u;
     RingGeom g;
     g.stage_bytes = uint32_t(3 * W) * es;
     g.stage_stride = (g.stage_bytes + align - 1) & ~(align - 1);
-    g.out_bytes = uint32_t(16 * (3 * (W / 8)));
+    g.out_bytes = uint32_t(4 * out_es * (3 * (W / 8)));
     return g;
 }
 
@@ -114,8 +114,9 @@ aol_status_t encode_row_map(CUtensorMap* map, aol_dtype_t dt, const void* base, 
 
 }  // namespace
 
-aol_status_t plan_fused(aol_dtype_t in_dtype, const void* d_in, const int32_t* d_out, int64_t frames,
-                        int64_t channels, int64_t H, int64_t W, const aol_launch_opts_t* opts, FusedPlan* plan) {
+aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void* d_in, const void* d_out,
+                        int64_t frames, int64_t channels, int64_t H, int64_t W, const aol_launch_opts_t* opts,
+                        FusedPlan* plan) {
     DeviceInfo dev;
     aol_status_t st = device_info(&dev);
     if (st != AOL_OK) return st;
@@ -124,10 +125,12 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, const void* d_in, const int32_t* d
     const int64_t Wo = 3 * (W / 8);
     *plan = FusedPlan{};
     plan->num_sms = dev.num_sms;
+    plan->out_es = out_dtype == AOL_I16 ? 2 : 4;
 
     bool tma_ok = tma_shape_ok(in_dtype, planes, channels, H, W) && (d_in == nullptr || aligned16(d_in)) &&
                   (d_out == nullptr || aligned16(d_out));
-    const RingGeom geom = ring_geom(in_dtype, W);
+    const int out_es = out_dtype == AOL_I16 ? 2 : 4;
+    const RingGeom geom = ring_geom(in_dtype, out_es, W);
     // repetitions per consumer thread: 2 for uint8 frames at least 1024 wide (HD: 0.498 vs 0.520 ms; 4K: equal),
     // 1 for narrower ones (CIF: 0.361 vs 0.315 ms -- one half-idle warp per CTA) and for int32
     // (profiles/r01_u8_r2_ab.jsonl)
@@ -141,9 +144,10 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, const void* d_in, const int32_t* d
         // concurrent row streams than that: DRAM efficiency falls as streams are added.  int32
         // (HBM-bound): 8 consumer warps per SM.  uint8 (issue-bound): 16 warps of one repetition each,
         // or 8 warps of two (HD: 2 CTAs/SM, 0.499 ms vs 0.567 at 3 and 0.738 at 1;
-        // profiles/r01_u8_r2_ab.jsonl).
+        // profiles/r01_u8_r2_ab.jsonl) -- 12 with int16 outputs, whose halved write traffic leaves DRAM room
+        // for a third row stream per SM (HD: 0.431 ms at 3 CTAs/SM vs 0.503 at 2; profiles/r01_u8_i16.jsonl).
         const int cwarps = nc / 32;
-        const int want_warps = (in_dtype == AOL_U8 && kr == 1) ? 16 : 8;
+        const int want_warps = (in_dtype == AOL_U8 && kr == 1) ? 16 : (in_dtype == AOL_U8 && out_es == 2) ? 12 : 8;
         cps = o.ctas_per_sm > 0 ? o.ctas_per_sm
                                 : std::max(1, std::min(8, (want_warps + cwarps - 1) / cwarps));
         for (;; --cps) {
@@ -159,8 +163,8 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, const void* d_in, const int32_t* d
             int occ = 0;
             const int smem = smem_bytes(geom, stages);
             if (stages >= 2 && cps > 1)
-                occ = kernel_occupancy(reinterpret_cast<const void*>(pick(in_dtype, true, kr, W, block, cps)), block,
-                                       smem);
+                occ = kernel_occupancy(reinterpret_cast<const void*>(pick(in_dtype, out_es, true, kr, W, block, cps)),
+                                       block, smem);
             if (cps == 1) occ = 1;   // one CTA always fits once its shared memory does
             if ((stages >= 2 && occ >= cps) || cps == 1 || o.ctas_per_sm > 0) {
                 if (stages < 2) tma_ok = false;
@@ -220,21 +224,25 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, const void* d_in, const int32_t* d
     return AOL_OK;
 }
 
-aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t in_dtype, int32_t* d_out,
+aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t in_dtype, void* d_out,
                           int64_t frames, int64_t channels, int64_t H, int64_t W, uint64_t* d_cs, cudaStream_t s) {
     const int64_t planes = frames * channels;
     const int32_t Ho = int32_t(4 * (H / 9)), Wo = int32_t(3 * (W / 8));
 
     if (plan.kernel == 2) {
         if (d_cs) AOL_CUDA_TRY(cudaMemsetAsync(d_cs, 0, size_t(frames) * sizeof(uint64_t), s));
-        if (in_dtype == AOL_U8) {
-            auto k = d_cs ? fused_generic_kernel<uint8_t, true> : fused_generic_kernel<uint8_t, false>;
-            k<<<plan.grid, plan.block, 0, s>>>(static_cast<const uint8_t*>(d_in), d_out, d_cs, planes, int32_t(H),
-                                               int32_t(W), Ho, Wo, int32_t(channels));
+        if (in_dtype == AOL_U8 && plan.out_es == 2) {
+            auto k = d_cs ? fused_generic_kernel<uint8_t, int16_t, true> : fused_generic_kernel<uint8_t, int16_t, false>;
+            k<<<plan.grid, plan.block, 0, s>>>(static_cast<const uint8_t*>(d_in), static_cast<int16_t*>(d_out), d_cs,
+                                               planes, int32_t(H), int32_t(W), Ho, Wo, int32_t(channels));
+        } else if (in_dtype == AOL_U8) {
+            auto k = d_cs ? fused_generic_kernel<uint8_t, int32_t, true> : fused_generic_kernel<uint8_t, int32_t, false>;
+            k<<<plan.grid, plan.block, 0, s>>>(static_cast<const uint8_t*>(d_in), static_cast<int32_t*>(d_out), d_cs,
+                                               planes, int32_t(H), int32_t(W), Ho, Wo, int32_t(channels));
         } else {
-            auto k = d_cs ? fused_generic_kernel<int32_t, true> : fused_generic_kernel<int32_t, false>;
-            k<<<plan.grid, plan.block, 0, s>>>(static_cast<const int32_t*>(d_in), d_out, d_cs, planes, int32_t(H),
-                                               int32_t(W), Ho, Wo, int32_t(channels));
+            auto k = d_cs ? fused_generic_kernel<int32_t, int32_t, true> : fused_generic_kernel<int32_t, int32_t, false>;
+            k<<<plan.grid, plan.block, 0, s>>>(static_cast<const int32_t*>(d_in), static_cast<int32_t*>(d_out), d_cs,
+                                               planes, int32_t(H), int32_t(W), Ho, Wo, int32_t(channels));
         }
         AOL_LAUNCH_CHECK("fused_generic_kernel");
         return AOL_OK;
@@ -269,7 +277,7 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
     a.bands_per_unit = plan.bands_per_unit;
     a.units_per_plane = plan.units_per_plane;
     a.stages = plan.stages;
-    const RingGeom geom = ring_geom(in_dtype, W);
+    const RingGeom geom = ring_geom(in_dtype, plan.out_es, W);
     a.stage_bytes = geom.stage_bytes;
     a.stage_stride = geom.stage_stride;
     a.out_bytes = geom.out_bytes;
@@ -278,7 +286,7 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
     a.hint_stores = (plan.flags & AOL_FLAG_EVICT_FIRST_STORES) ? 1 : 0;
     a.blocked_units = (plan.flags & AOL_FLAG_BLOCKED_UNITS) ? 1 : 0;
 
-    KernelFn k = pick(in_dtype, d_cs != nullptr, plan.reps_per_thread, W, plan.block, plan.ctas_per_sm);
+    KernelFn k = pick(in_dtype, plan.out_es, d_cs != nullptr, plan.reps_per_thread, W, plan.block, plan.ctas_per_sm);
     aol_status_t st_attr = kernel_smem(reinterpret_cast<const void*>(k), plan.smem);
     if (st_attr != AOL_OK) return st_attr;
     // With checksums: zero them in a one-CTA kernel and launch the fused kernel as its programmatic

@@ -11,12 +11,20 @@ KernelFn tma_kernel_u8_cs(int block, int cps);
 KernelFn tma_kernel_u8_nocs(int block, int cps);
 KernelFn tma_kernel_u8r2_cs(int block, int cps);
 KernelFn tma_kernel_u8r2_nocs(int block, int cps);
+KernelFn tma_kernel_u8h_cs(int block, int cps);
+KernelFn tma_kernel_u8h_nocs(int block, int cps);
+KernelFn tma_kernel_u8r2h_cs(int block, int cps);
+KernelFn tma_kernel_u8r2h_nocs(int block, int cps);
 
 KernelFn tma_kernel_i32(bool checksum, bool swz32, int block, int cps) {
     if (swz32) return checksum ? tma_kernel_i32s_cs(block, cps) : tma_kernel_i32s_nocs(block, cps);
     return checksum ? tma_kernel_i32_cs(block, cps) : tma_kernel_i32_nocs(block, cps);
 }
-KernelFn tma_kernel_u8(bool checksum, int reps_per_thread, int block, int cps) {
+KernelFn tma_kernel_u8(bool checksum, bool out16, int reps_per_thread, int block, int cps) {
+    if (out16) {
+        if (reps_per_thread == 2) return checksum ? tma_kernel_u8r2h_cs(block, cps) : tma_kernel_u8r2h_nocs(block, cps);
+        return checksum ? tma_kernel_u8h_cs(block, cps) : tma_kernel_u8h_nocs(block, cps);
+    }
     if (reps_per_thread == 2) return checksum ? tma_kernel_u8r2_cs(block, cps) : tma_kernel_u8r2_nocs(block, cps);
     return checksum ? tma_kernel_u8_cs(block, cps) : tma_kernel_u8_nocs(block, cps);
 }

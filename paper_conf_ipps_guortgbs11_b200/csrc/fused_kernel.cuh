@@ -82,7 +82,7 @@ __device__ __forceinline__ int32_t task_T_small(int32_t S) {
 }
 
 struct FusedArgs {
-    int32_t* Z;
+    void* Z;                    // output, Tout elements (int32, or int16 for 8-bit samples)
     uint64_t* cs;
     const void* X;              // uint8 path: source of the 1-D bulk copies
     int64_t nunits;
@@ -97,7 +97,7 @@ struct FusedArgs {
     int32_t stages;
     uint32_t stage_bytes;   // bytes of one row triple (12W int32, 3W uint8)
     uint32_t stage_stride;  // stage_bytes rounded up (1024 for the swizzle atom, 128 for uint8)
-    uint32_t out_bytes;     // 16*Wo  (4 output rows)
+    uint32_t out_bytes;     // 4 output rows: 4 * Wo * sizeof(Tout)
     int32_t n_consumer;     // consumer threads, multiple of 32
     int32_t hint_loads;     // 1: TMA loads with L2 evict_first (input is streamed once)
     int32_t hint_stores;    // 1: bulk stores with L2 evict_first
@@ -202,8 +202,8 @@ __device__ __forceinline__ void h_row(uint32_t row_base, uint32_t rr, const RepG
 // 8 columns); 1 or 2 for uint8 input, whose 16 bytes for two repetitions come in one LDS.128 and whose per-stage
 // bookkeeping (mbarrier wait/arrive, addressing) two repetitions then share (the host picks, fused.cu).
 // kSwz = the int32 smem layout: 128 (SWIZZLE_128B, W % 32 == 0) or 32 (SWIZZLE_32B, other W % 8 == 0);
-// unused (0) for uint8.
-template <typename Tin, int kR, int kSwz, bool kChecksum, int kMaxThreads, int kMinBlocks>
+// unused (0) for uint8.  Tout = output element: int32, or int16 for 8-bit samples (outputs in [-5, 255]).
+template <typename Tin, typename Tout, int kR, int kSwz, bool kChecksum, int kMaxThreads, int kMinBlocks>
 __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
     fused_tma_kernel(const __grid_constant__ CUtensorMap tmap, const FusedArgs a) {
     constexpr bool kI32 = std::is_same<Tin, int32_t>::value;
@@ -211,7 +211,7 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
     extern __shared__ uint8_t smem_raw[];
     uint8_t* smem = reinterpret_cast<uint8_t*>((reinterpret_cast<uintptr_t>(smem_raw) + 1023) & ~uintptr_t(1023));
     uint8_t* stage_base = smem;
-    int32_t* outbuf = reinterpret_cast<int32_t*>(smem + size_t(a.stages) * a.stage_stride);
+    uint8_t* outbuf = smem + size_t(a.stages) * a.stage_stride;
     uint64_t* full = reinterpret_cast<uint64_t*>(smem + size_t(a.stages) * a.stage_stride + kOutBufs * a.out_bytes);
     uint64_t* empty = full + a.stages;
     unsigned long long* red = reinterpret_cast<unsigned long long*>(empty + a.stages);   // [32] checksum partials
@@ -336,26 +336,34 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
             const uint32_t ob = ptx::smem_u32(outbuf) + (emit_idx % kOutBufs) * a.out_bytes;
             if (active) {
 #pragma unroll
-                for (int k = 0; k < 4; ++k)
+                for (int k = 0; k < 4; ++k) {
+                    const uint32_t e0 = uint32_t(k * Wo + 3 * r);   // element index of the thread's first column
+                    if constexpr (sizeof(Tout) == 4 && kR == 1) {
 #pragma unroll
-                    if constexpr (kR == 1) {
+                        for (int m = 0; m < 3; ++m) ptx::sts32(ob + 4u * (e0 + m), z[k][m]);
+                    } else if constexpr (sizeof(Tout) == 4) {   // 8-byte aligned pairs: Wo = 6 (W/16) and 3r even
 #pragma unroll
-                        for (int m = 0; m < 3; ++m) ptx::sts32(ob + 4u * uint32_t(k * Wo + 3 * r + m), z[k][m]);
-                    } else {   // 8-byte aligned pairs: Wo = 6 (W/16) and 3r are even
+                        for (int m = 0; m < kC; m += 2) ptx::sts64(ob + 4u * (e0 + m), z[k][m], z[k][m + 1]);
+                    } else if constexpr (kR == 1) {             // int16
+#pragma unroll
+                        for (int m = 0; m < 3; ++m) ptx::sts16(ob + 2u * (e0 + m), z[k][m]);
+                    } else {   // int16 pairs packed into 32-bit stores (e0 even)
 #pragma unroll
                         for (int m = 0; m < kC; m += 2)
-                            ptx::sts64(ob + 4u * uint32_t(k * Wo + 3 * r + m), z[k][m], z[k][m + 1]);
+                            ptx::sts32(ob + 2u * (e0 + m),
+                                       int32_t((uint32_t(z[k][m]) & 0xffffu) | (uint32_t(z[k][m + 1]) << 16)));
                     }
+                }
             }
             ptx::fence_proxy_async_smem();
             ptx::named_bar_sync(1, NC);
             if (tid == 0) {
-                int32_t* gz = a.Z + (size_t(plane) * a.Ho + size_t(4 * band)) * size_t(Wo);
+                Tout* gz = static_cast<Tout*>(a.Z) + (size_t(plane) * a.Ho + size_t(4 * band)) * size_t(Wo);
+                const uint8_t* src = outbuf + (emit_idx % kOutBufs) * a.out_bytes;
                 if (a.hint_stores)
-                    ptx::bulk_store_hint(gz, outbuf + (emit_idx % kOutBufs) * (a.out_bytes / 4), a.out_bytes,
-                                         ptx::policy_evict_first());
+                    ptx::bulk_store_hint(gz, src, a.out_bytes, ptx::policy_evict_first());
                 else
-                    ptx::bulk_store(gz, outbuf + (emit_idx % kOutBufs) * (a.out_bytes / 4), a.out_bytes);   // 4 rows
+                    ptx::bulk_store(gz, src, a.out_bytes);   // 4 rows
                 ptx::bulk_commit();
             }
             ++emit_idx;
@@ -468,9 +476,9 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
 // One thread per (plane, band, output column): recomputes the 12 Y values it
 // needs straight from global memory (L1/L2 absorb the overlap).  Correct for
 // every shape; used when the TMA kernel's geometry constraints do not hold.
-template <typename Tin, bool kChecksum>
+template <typename Tin, typename Tout, bool kChecksum>
 __global__ void __launch_bounds__(256)
-    fused_generic_kernel(const Tin* __restrict__ X, int32_t* __restrict__ Z, uint64_t* __restrict__ cs,
+    fused_generic_kernel(const Tin* __restrict__ X, Tout* __restrict__ Z, uint64_t* __restrict__ cs,
                          int64_t planes, int32_t H, int32_t W, int32_t Ho, int32_t Wo, int32_t channels) {
     const int32_t nb = H / 9;
     const int64_t total = planes * nb * int64_t(Wo);
@@ -508,7 +516,7 @@ __global__ void __launch_bounds__(256)
                 for (int t = 0; t < 6; ++t) S += int32_t(xr[col[t]]);
                 yv[j] = task_T(S);
             }
-            int32_t* Zp = Z + size_t(plane) * Ho * Wo;
+            Tout* Zp = Z + size_t(plane) * Ho * Wo;
             const int32_t chan = int32_t(plane % channels);
 #pragma unroll
             for (int kk = 0; kk < 4; ++kk) {
@@ -517,7 +525,7 @@ __global__ void __launch_bounds__(256)
                 for (int t = 0; t < 6; ++t) S += yv[2 * kk + t];
                 const int32_t z = task_T(S);
                 const int32_t yo = 4 * b + kk;
-                Zp[size_t(yo) * Wo + xo] = z;
+                Zp[size_t(yo) * Wo + xo] = Tout(z);
                 if (kChecksum)
                     contrib += uint64_t(uint32_t(z)) * (1u + (uint64_t(chan) * Ho + yo) * uint64_t(Wo) + xo);
             }
@@ -542,22 +550,22 @@ using KernelFn = void (*)(const CUtensorMap, const FusedArgs);
 
 // Explicit instantiations live in fused_k_*.cu (compiled in parallel); these pick one.
 KernelFn tma_kernel_i32(bool checksum, bool swz32, int block, int cps);
-KernelFn tma_kernel_u8(bool checksum, int reps_per_thread, int block, int cps);
+KernelFn tma_kernel_u8(bool checksum, bool out16, int reps_per_thread, int block, int cps);
 
-template <typename Tin, int kR, int kSwz, bool kChecksum>
+template <typename Tin, typename Tout, int kR, int kSwz, bool kChecksum>
 KernelFn pick_tma_kernel(int block, int cps) {
     if constexpr (kR == 2) {
         // two repetitions per thread take ~126 registers: bounds that never force spills below 1024 threads
-        if (block <= 160 && cps >= 3) return fused_tma_kernel<Tin, kR, kSwz, kChecksum, 160, 3>;
-        if (block <= 256 && cps >= 2) return fused_tma_kernel<Tin, kR, kSwz, kChecksum, 256, 2>;
-        if (block <= 512) return fused_tma_kernel<Tin, kR, kSwz, kChecksum, 512, 1>;
-        return fused_tma_kernel<Tin, kR, kSwz, kChecksum, 1024, 1>;
+        if (block <= 160 && cps >= 3) return fused_tma_kernel<Tin, Tout, kR, kSwz, kChecksum, 160, 3>;
+        if (block <= 256 && cps >= 2) return fused_tma_kernel<Tin, Tout, kR, kSwz, kChecksum, 256, 2>;
+        if (block <= 512) return fused_tma_kernel<Tin, Tout, kR, kSwz, kChecksum, 512, 1>;
+        return fused_tma_kernel<Tin, Tout, kR, kSwz, kChecksum, 1024, 1>;
     } else {
-        if (block <= 128 && cps >= 3) return fused_tma_kernel<Tin, kR, kSwz, kChecksum, 128, 4>;
-        if (block <= 320 && cps >= 3) return fused_tma_kernel<Tin, kR, kSwz, kChecksum, 320, 3>;
-        if (block <= 320 && cps >= 2) return fused_tma_kernel<Tin, kR, kSwz, kChecksum, 320, 2>;
-        if (block <= 512) return fused_tma_kernel<Tin, kR, kSwz, kChecksum, 512, 1>;
-        return fused_tma_kernel<Tin, kR, kSwz, kChecksum, 1024, 1>;
+        if (block <= 128 && cps >= 3) return fused_tma_kernel<Tin, Tout, kR, kSwz, kChecksum, 128, 4>;
+        if (block <= 320 && cps >= 3) return fused_tma_kernel<Tin, Tout, kR, kSwz, kChecksum, 320, 3>;
+        if (block <= 320 && cps >= 2) return fused_tma_kernel<Tin, Tout, kR, kSwz, kChecksum, 320, 2>;
+        if (block <= 512) return fused_tma_kernel<Tin, Tout, kR, kSwz, kChecksum, 512, 1>;
+        return fused_tma_kernel<Tin, Tout, kR, kSwz, kChecksum, 1024, 1>;
     }
 }
 

@@ -76,6 +76,10 @@ __device__ __forceinline__ void griddep_launch_dependents() {
     asm volatile("griddepcontrol.launch_dependents;" ::: "memory");
 }
 
+__device__ __forceinline__ void sts16(uint32_t saddr, int32_t v) {
+    asm volatile("st.shared.b16 [%0], %1;" ::"r"(saddr), "h"(static_cast<unsigned short>(v)) : "memory");
+}
+
 __device__ __forceinline__ void sts64(uint32_t saddr, int32_t a, int32_t b) {
     asm volatile("st.shared.v2.s32 [%0], {%1, %2};" ::"r"(saddr), "r"(a), "r"(b) : "memory");
 }

@@ -188,6 +188,37 @@ def test_fused_u8_two_reps_per_thread(orc, W):
         assert plan["block"] == ((W // 8 // kr) + 31) // 32 * 32 + 32, (flags, plan)
 
 
+@pytest.mark.parametrize("shape,kernel", [
+    ((1, 3, 1080, 1920), 1), ((2, 3, 288, 352), 1), ((2, 3, 36, 1040), 1), ((2, 3, 36, 128), 1),
+    ((1, 2, 18, 40), 2), ((2, 3, 36, 128), 2),
+])
+def test_fused_u8_int16_output(orc, shape, kernel):
+    """NEXT row f1's int16 output option: 8-bit samples give outputs in [-5, 255]; stored as int16 they are
+    the oracle's integers, and the checksums equal the int32-output run's."""
+    N, C, H, W = shape
+    xh = synth.frames(25, 0, N, C, H, W, "uniform")
+    xh[0, 0] = synth.frames(26, 0, 1, 1, H, W, "dark")[0, 0]   # negative outputs on one plane
+    zo, cso = run_oracle(orc, xh)
+    x8 = torch.from_numpy(xh.astype(np.uint8)).cuda()
+    opts = {"kernel": kernel}
+    plan = aol.downscale_frame_plan(N, C, H, W, dtype=torch.uint8, opts=opts, out_dtype=torch.int16)
+    assert plan["kernel"] == kernel
+    z, cs = aol.downscale_frame(x8, checksums=True, opts=opts, out_dtype=torch.int16)
+    z2, _ = aol.downscale_frame(x8, opts=opts, out_dtype=torch.int16)
+    torch.cuda.synchronize()
+    assert z.dtype == torch.int16
+    assert np.array_equal(z.cpu().numpy().astype(np.int32), zo)
+    assert np.array_equal(z2.cpu().numpy().astype(np.int32), zo)
+    assert np.array_equal(np_u64(cs), cso)
+
+
+def test_int16_output_needs_uint8_input():
+    x = torch.zeros((1, 1, 9, 32), dtype=torch.int32, device="cuda")
+    with pytest.raises(aol.AolError) as e:
+        aol.downscale_frame(x, out_dtype=torch.int16)
+    assert e.value.status == aol._lib.E_DTYPE
+
+
 def test_no_checksum_and_zero_frames(orc):
     xh = synth.frames(1, 0, 1, 3, 18, 64)
     z, cs = aol.downscale_frame(torch.from_numpy(xh).cuda())

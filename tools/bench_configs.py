@@ -56,18 +56,19 @@ def emit(d):
     print(json.dumps(d), flush=True)
 
 
-def frames_bytes(N, C, H, W, es=4):
-    return N * C * (H * W * es + (4 * (H // 9)) * (3 * (W // 8)) * 4)
+def frames_bytes(N, C, H, W, es=4, eo=4):
+    return N * C * (H * W * es + (4 * (H // 9)) * (3 * (W // 8)) * eo)
 
 
-def fused_line(name, N, C, H, W, dtype=torch.int32, opts=None, reps=20):
+def fused_line(name, N, C, H, W, dtype=torch.int32, opts=None, reps=20, out_dtype=torch.int32):
     x = aol.synth_frames(3, 0, N, C, H, W, "uniform", dtype=dtype)
-    z = torch.empty((N, C, 4 * (H // 9), 3 * (W // 8)), dtype=torch.int32, device="cuda")
+    z = torch.empty((N, C, 4 * (H // 9), 3 * (W // 8)), dtype=out_dtype, device="cuda")
     cs = torch.empty(N, dtype=torch.uint64, device="cuda")
     med, mn = timed(lambda: aol.downscale_frame(x, out=z, checksums=cs, opts=opts), reps=reps)
-    b = frames_bytes(N, C, H, W, x.element_size())
-    plan = aol.downscale_frame_plan(N, C, H, W, dtype=dtype, opts=opts)
-    emit({"config": name, "shape": [N, C, H, W], "dtype": str(dtype).split(".")[-1], "ms": med, "min_ms": mn,
+    b = frames_bytes(N, C, H, W, x.element_size(), z.element_size())
+    plan = aol.downscale_frame_plan(N, C, H, W, dtype=dtype, opts=opts, out_dtype=out_dtype)
+    emit({"config": name, "shape": [N, C, H, W], "dtype": str(dtype).split(".")[-1],
+          "out_dtype": str(out_dtype).split(".")[-1], "ms": med, "min_ms": mn,
           "frames_per_s": N / (med / 1e3), "GBps": b / (med / 1e3) / 1e9, "frac": b / (med / 1e3) / 1e9 / peak(),
           "kernel": plan["kernel"], "plan": plan})
     del x, z, cs
@@ -191,6 +192,7 @@ def main():
         fused_line("d4 4K batch", 64, 3, 2160, 3840)
     if want("f1"):
         fused_line("f1 HD uint8 input", 300, 3, 1080, 1920, dtype=torch.uint8)
+        fused_line("f1 HD uint8 input, int16 output", 300, 3, 1080, 1920, dtype=torch.uint8, out_dtype=torch.int16)
     if want("f4"):
         fused_line("f4 CIF 2000 frames", 2000, 3, 288, 352)
 
