@@ -209,7 +209,9 @@ __global__ void __launch_bounds__(256) tiler_linear32_kernel(const TilerDev td, 
     __syncthreads();
     const int32_t nvec = int32_t(td.total / V);
     const int32_t stride = int32_t(gridDim.x * blockDim.x);
-    constexpr int kU = 4;
+    // 2 vectors per thread per iteration with a 4x larger grid than the general kernels (tools/tiler_probe2.py,
+    // profiles/r01_tiler_variants.jsonl: d3 gather 5.01 -> 5.22 TB/s; kU = 1, 4, 8 and grids x8..x512 are slower)
+    constexpr int kU = 2;
     const int32_t warp_first = int32_t((blockIdx.x * blockDim.x + (threadIdx.x & ~31u)) * kU + (threadIdx.x & 31u));
     for (int32_t v0 = warp_first; v0 < nvec; v0 += kU * stride) {
         int32_t off[kU], g[kU];
@@ -258,7 +260,11 @@ aol_status_t launch_v(const TilerDev& td, const void* src, void* dst, unsigned l
                       cudaStream_t s) {
     const bool fast = td.fast32 != 0, lin = td.linear != 0;
     if (MODE <= 1 && lin && td.small32) {
-        tiler_linear32_kernel<ES, V, MODE><<<grid, 256, 0, s>>>(td, src, dst);
+        DeviceInfo dev;
+        aol_status_t st = device_info(&dev);
+        if (st != AOL_OK) return st;
+        const int g32 = int(std::max<int64_t>(1, std::min<int64_t>((td.total / V + 255) / 256, int64_t(dev.num_sms) * 128)));
+        tiler_linear32_kernel<ES, V, MODE><<<g32, 256, 0, s>>>(td, src, dst);
         AOL_LAUNCH_CHECK("tiler_linear32_kernel");
         return AOL_OK;
     }
