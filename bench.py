@@ -58,6 +58,8 @@ def parse():
     p.add_argument("--e2e-steps", type=int, default=3)
     p.add_argument("--no-e2e", action="store_true")
     p.add_argument("--no-cpu-baseline", action="store_true")
+    p.add_argument("--cpu-baseline-seconds", type=float, default=10.0,
+                   help="wall time the cpu_baseline leg spends re-running its sample (median pass reported)")
     p.add_argument("--dump-checksums", type=str, default="",
                    help="rank 0 saves the gathered per-frame checksums (global frame order, .npy) for the tests")
     return p.parse_args()
@@ -165,10 +167,12 @@ class ClockSampler:
                 "reasons": sorted(self.reasons), "samples": len(self.samples)}
 
 
-def cpu_baseline(a, gpu_cs=None, frame0=0, steps=1):
+def cpu_baseline(a, gpu_cs=None, frame0=0, steps=1, min_seconds=0.0):
     """Time the CPU oracle (as it stands, OpenMP across planes) on a bounded sample.
-    Returns (frames_per_s, info).  Also checks oracle checksums against the GPU's for
-    the unique sample frames when gpu_cs is given."""
+    At least `steps` passes over the sample, and more until `min_seconds` of wall time
+    have been spent (so the sample is ~10 s of work however many cores the host has).
+    Returns (frames_per_s, info): the median pass rate.  Also checks oracle checksums
+    against the GPU's for the unique sample frames when gpu_cs is given."""
     import numpy as np
 
     import oracle
@@ -186,14 +190,14 @@ def cpu_baseline(a, gpu_cs=None, frame0=0, steps=1):
     oracle.downscale_frame(x[:1], nthreads=1)  # warm the library
     times = []
     cs = None
-    for _ in range(steps):
+    while len(times) < steps or sum(times) < min_seconds:
         t0 = time.perf_counter()
         _, cs = oracle.downscale_frame(x, nthreads=nthreads)
         times.append(time.perf_counter() - t0)
     dt = statistics.median(times)
     info = {"cores": nthreads, "sample": f"{sample} frames of the workload ({uniq} unique, seed {a.seed}, "
                                         f"frames {frame0}..{frame0 + uniq - 1} repeated), OpenMP over planes, "
-                                        f"median of {steps}", "seconds": dt}
+                                        f"median pass of {len(times)} ({sum(times):.1f} s wall)", "seconds": dt}
     if gpu_cs is not None:
         info["parity_sample_ok"] = bool(np.array_equal(cs[:uniq], gpu_cs[:uniq]))
     return sample / dt, info
@@ -388,7 +392,8 @@ def main():
     if world > 1 and cs_all is not None:
         line["gathered_checksums"] = int(cs_all.size)
     if world == 1 and not a.no_cpu_baseline:
-        fps, info = cpu_baseline(a, gpu_cs=cs.cpu().view(torch.int64).numpy().view(np.uint64), frame0=frame0)
+        fps, info = cpu_baseline(a, gpu_cs=cs.cpu().view(torch.int64).numpy().view(np.uint64), frame0=frame0,
+                                 min_seconds=a.cpu_baseline_seconds)
         line["cpu_baseline"] = {"value": fps, "unit": "frames/s", "cores": info["cores"], "kind": "oracle",
                                 "sample": info["sample"], "parity_sample_ok": info.get("parity_sample_ok")}
     print(json.dumps(line), flush=True)

@@ -117,6 +117,10 @@ typedef struct {
                                           (default: overlapped, programmatic dependent launch)        */
 #define AOL_FLAG_U8_ONE_REP 32         /* uint8 input: one H repetition per consumer thread even for
                                           W >= 1024 (default there: two)                            */
+#define AOL_FLAG_I32_LINEAR 128        /* int32 input: 1-D bulk copies into linear smem rows even when
+                                          W % 32 == 0 (default there: TMA tensor loads, SWIZZLE_128B) */
+#define AOL_FLAG_I32_SWZ32 256         /* int32 input, W % 32 != 0, W <= 2048: TMA tensor loads of
+                                          32-byte lines under SWIZZLE_32B (default: linear rows)     */
 
 /* The launch configuration aol_downscale_frame_ex would use (for reports/tests). */
 typedef struct {

@@ -47,24 +47,36 @@ aol_status_t get_encode_fn(EncodeTiledFn* fn) {
     return AOL_OK;
 }
 
-bool tma_shape_ok(aol_dtype_t dt, int64_t planes, int64_t channels, int64_t H, int64_t W) {
+// Shared-memory layout of an int32 row triple (the kernel's kSwz): 128 = TMA tensor loads of 128-byte lines
+// under SWIZZLE_128B (W % 32 == 0); 0 = one 1-D bulk copy of the contiguous triple into linear rows (W % 32 != 0,
+// or forced by AOL_FLAG_I32_LINEAR); 32 = TMA tensor loads of 32-byte lines under SWIZZLE_32B (W % 32 != 0 with
+// AOL_FLAG_I32_SWZ32, W <= 2048: the round-1 layout, kept for A/B).  -1 for uint8 input.
+int i32_layout(aol_dtype_t dt, int64_t W, int flags) {
+    if (dt != AOL_I32) return -1;
+    if (flags & AOL_FLAG_I32_LINEAR) return 0;
+    if (W % 32 == 0) return 128;
+    return (flags & AOL_FLAG_I32_SWZ32) ? 32 : 0;
+}
+
+bool tma_shape_ok(aol_dtype_t dt, int64_t planes, int64_t channels, int64_t H, int64_t W, int flags) {
     if (H < 9 || W / 8 > kMaxConsumers) return false;
     // checksum weights (1 + frame-local output index) are computed in 32 bits
     if (channels * (4 * (H / 9)) * (3 * (W / 8)) >= (int64_t(1) << 32) - 1) return false;
-    // int32: {32, W/32, 3}-element boxes under SWIZZLE_128B, or {8, W/8, 3} under SWIZZLE_32B when W % 32 != 0
-    // (a box dimension holds at most 256 elements)
-    if (dt == AOL_I32)
-        return (W % 32 == 0 ? W / 32 <= 256 : W / 8 <= 256) && planes * H < (int64_t(1) << 31);
+    // int32 tensor layouts: {32, W/32, 3}-element boxes under SWIZZLE_128B or {8, W/8, 3} under SWIZZLE_32B
+    // (a box dimension holds at most 256 elements; tensor row coordinates are int32); linear rows: 1-D bulk
+    // copies of 12W bytes (16-byte multiple since W % 8 == 0)
+    if (dt == AOL_I32) {
+        const int layout = i32_layout(dt, W, flags);
+        if (layout == 0) return true;
+        return (layout == 128 ? W / 32 <= 256 : W / 8 <= 256) && planes * H < (int64_t(1) << 31);
+    }
     if (dt == AOL_U8) return W % 16 == 0;   // 1-D bulk copies: 16-byte granularity
     return false;
 }
 
-// int32 frames whose width is not a multiple of 32 use 32-byte lines (SWIZZLE_32B)
-bool swz32_layout(aol_dtype_t dt, int64_t W) { return dt == AOL_I32 && W % 32 != 0; }
-
-KernelFn pick(aol_dtype_t dt, int out_es, bool checksum, int kr, int64_t W, int block, int cps) {
+KernelFn pick(aol_dtype_t dt, int out_es, bool checksum, int kr, int64_t W, int flags, int block, int cps) {
     return dt == AOL_U8 ? tma_kernel_u8(checksum, out_es == 2, kr, block, cps)
-                        : tma_kernel_i32(checksum, swz32_layout(dt, W), block, cps);
+                        : tma_kernel_i32(checksum, i32_layout(dt, W, flags), block, cps);
 }
 
 // Shared-memory geometry of the TMA ring: one stage = one row triple.
@@ -74,8 +86,9 @@ struct RingGeom {
     uint32_t out_bytes;     // one band of output: 4 rows of Wo output elements
 };
 
-RingGeom ring_geom(aol_dtype_t dt, int out_es, int64_t W) {
-    const uint32_t es = dt == AOL_U8 ? 1u : 4u, align = dt == AOL_U8 ? 128u : 1024u;
+RingGeom ring_geom(aol_dtype_t dt, int out_es, int64_t W, int flags) {
+    // swizzled layouts need 1024-byte aligned stages (the swizzle atom); bulk copies 16 bytes (128 kept)
+    const uint32_t es = dt == AOL_U8 ? 1u : 4u, align = i32_layout(dt, W, flags) > 0 ? 1024u : 128u;
     RingGeom g;
     g.stage_bytes = uint32_t(3 * W) * es;
     g.stage_stride = (g.stage_bytes + align - 1) & ~(align - 1);
@@ -90,12 +103,12 @@ int smem_bytes(const RingGeom& g, int stages) {
 
 // TMA descriptor for row triples of a [rows][W] array viewed as {inner, W/inner, rows}: int32 with a
 // 128 B swizzle (inner = 32 elements), uint8 unswizzled (inner = 128 elements).
-aol_status_t encode_row_map(CUtensorMap* map, aol_dtype_t dt, const void* base, int64_t rows, int64_t W) {
+aol_status_t encode_row_map(CUtensorMap* map, aol_dtype_t dt, const void* base, int64_t rows, int64_t W, int flags) {
     EncodeTiledFn encode;
     aol_status_t st = get_encode_fn(&encode);
     if (st != AOL_OK) return st;
     const bool i32 = dt == AOL_I32;
-    const bool s32 = swz32_layout(dt, W);
+    const bool s32 = i32_layout(dt, W, flags) == 32;
     const cuuint64_t inner = i32 ? (s32 ? 8 : 32) : 128, es = i32 ? 4 : 1;
     const cuuint64_t gdim[3] = {inner, cuuint64_t(W) / inner, cuuint64_t(rows)};
     const cuuint64_t gstride[2] = {inner * es, cuuint64_t(W) * es};
@@ -127,10 +140,10 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void*
     plan->num_sms = dev.num_sms;
     plan->out_es = out_dtype == AOL_I16 ? 2 : 4;
 
-    bool tma_ok = tma_shape_ok(in_dtype, planes, channels, H, W) && (d_in == nullptr || aligned16(d_in)) &&
+    bool tma_ok = tma_shape_ok(in_dtype, planes, channels, H, W, o.flags) && (d_in == nullptr || aligned16(d_in)) &&
                   (d_out == nullptr || aligned16(d_out));
     const int out_es = out_dtype == AOL_I16 ? 2 : 4;
-    const RingGeom geom = ring_geom(in_dtype, out_es, W);
+    const RingGeom geom = ring_geom(in_dtype, out_es, W, o.flags);
     // repetitions per consumer thread: 2 for uint8 frames at least 1024 wide (HD: 0.498 vs 0.520 ms; 4K: equal),
     // 1 for narrower ones (CIF: 0.361 vs 0.315 ms -- one half-idle warp per CTA) and for int32
     // (profiles/r01_u8_r2_ab.jsonl)
@@ -163,7 +176,7 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void*
             int occ = 0;
             const int smem = smem_bytes(geom, stages);
             if (stages >= 2 && cps > 1)
-                occ = kernel_occupancy(reinterpret_cast<const void*>(pick(in_dtype, out_es, true, kr, W, block, cps)),
+                occ = kernel_occupancy(reinterpret_cast<const void*>(pick(in_dtype, out_es, true, kr, W, o.flags, block, cps)),
                                        block, smem);
             if (cps == 1) occ = 1;   // one CTA always fits once its shared memory does
             if ((stages >= 2 && occ >= cps) || cps == 1 || o.ctas_per_sm > 0) {
@@ -174,8 +187,8 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void*
     }
     if (o.kernel == 1 && !tma_ok) {
         set_error("TMA fused kernel requested but unsupported for this shape/dtype/alignment "
-                  "(int32: W <= 7680 when W %% 32 == 0, else W <= 2048; uint8: W %% 16 == 0 and W <= 7936; "
-                  "16-byte aligned buffers)");
+                  "(W <= 7936 and a 2-stage ring within shared memory; int32 with W %% 32 == 0: W <= 7680; "
+                  "uint8: W %% 16 == 0; 16-byte aligned buffers)");
         return AOL_E_SHAPE;
     }
     if (o.kernel == 2) tma_ok = false;
@@ -252,8 +265,9 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
     std::memset(&map, 0, sizeof map);
     const bool u8_tensor = in_dtype == AOL_U8 && W % 128 == 0 && W / 128 <= 256 &&
                            planes * H < (int64_t(1) << 31) && !(plan.flags & AOL_FLAG_U8_BULK);
-    if (in_dtype == AOL_I32 || u8_tensor) {
-        aol_status_t st = encode_row_map(&map, in_dtype, d_in, planes * H, W);
+    const int layout = i32_layout(in_dtype, W, plan.flags);
+    if (layout > 0 || u8_tensor) {
+        aol_status_t st = encode_row_map(&map, in_dtype, d_in, planes * H, W, plan.flags);
         if (st != AOL_OK) return st;
     }
     FusedArgs a;
@@ -271,13 +285,13 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
     a.Wo = Wo;
     a.channels = int32_t(channels);
     a.reps = int32_t(W / 8);
-    a.segs = int32_t(swz32_layout(in_dtype, W) ? W / 8 : W / 32);   // int32 lines per row
+    a.segs = int32_t(layout == 32 ? W / 8 : W / 32);   // int32 swizzled lines per row (unused for linear rows)
     a.triples_per_plane = int32_t(H / 3);
     a.nbands = int32_t(H / 9);
     a.bands_per_unit = plan.bands_per_unit;
     a.units_per_plane = plan.units_per_plane;
     a.stages = plan.stages;
-    const RingGeom geom = ring_geom(in_dtype, plan.out_es, W);
+    const RingGeom geom = ring_geom(in_dtype, plan.out_es, W, plan.flags);
     a.stage_bytes = geom.stage_bytes;
     a.stage_stride = geom.stage_stride;
     a.out_bytes = geom.out_bytes;
@@ -286,7 +300,8 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
     a.hint_stores = (plan.flags & AOL_FLAG_EVICT_FIRST_STORES) ? 1 : 0;
     a.blocked_units = (plan.flags & AOL_FLAG_BLOCKED_UNITS) ? 1 : 0;
 
-    KernelFn k = pick(in_dtype, plan.out_es, d_cs != nullptr, plan.reps_per_thread, W, plan.block, plan.ctas_per_sm);
+    KernelFn k = pick(in_dtype, plan.out_es, d_cs != nullptr, plan.reps_per_thread, W, plan.flags, plan.block,
+                      plan.ctas_per_sm);
     aol_status_t st_attr = kernel_smem(reinterpret_cast<const void*>(k), plan.smem);
     if (st_attr != AOL_OK) return st_attr;
     // With checksums: zero them in a one-CTA kernel and launch the fused kernel as its programmatic

@@ -20,7 +20,9 @@
 //    round-robin.
 //  * One producer warp fills an S-stage smem ring guarded by full/empty
 //    mbarriers.  int32 input: 3-D TMA tensor loads (box = 3 rows x W,
-//    SWIZZLE_128B).  uint8 input ("24-bit RGB"): 3-D TMA tensor loads of
+//    SWIZZLE_128B) when W % 32 == 0, else 1-D TMA bulk copies of the contiguous
+//    3-row triple into a linear layout read conflict-free by lane-rotated
+//    LDS.128 (kSwz = 0).  uint8 input ("24-bit RGB"): 3-D TMA tensor loads of
 //    {128 B, W/128, 3 rows} without swizzle when W % 128 == 0, else 1-D TMA bulk
 //    copies of the contiguous 3-row triple (same smem layout either way).
 //  * Consumer thread r owns repetition r (8 input columns -> 3 Y columns).
@@ -128,10 +130,12 @@ __device__ __forceinline__ int64_t unit_of(const FusedArgs& a, int64_t k) {
 
 // Per-thread constants of the H stage (which repetition, where its bytes live).
 struct RepGeom {
-    uint32_t off0, off1;  // int32: swizzled offsets of the two chunks within a row's lines; uint8: 8r
+    uint32_t off0, off1;  // int32: swizzled offsets of the two chunks within a row's lines (kSwz = 0: byte
+                          // offsets of the first / second chunk LOADED); uint8: 8r
     uint32_t offn;        // neighbour repetition's first chunk / word
     uint32_t seg, segn;   // int32: 128-byte segment (32-byte line with kSwz == 32) of the repetition / neighbour
     bool fix;             // read the neighbour from smem instead of the shuffle
+    bool swap;            // int32, kSwz = 0: the thread loads its upper chunk first (bank rotation)
 };
 
 // H stage of one input row: the three 6-tap window sums of each of the thread's kR repetitions, T() applied:
@@ -143,7 +147,16 @@ __device__ __forceinline__ void h_row(uint32_t row_base, uint32_t rr, const RepG
         static_assert(kR == 1, "int32 path: one repetition per thread");
         const uint32_t line = rr * segs + g.seg;
         int4 q0, q1;
-        if constexpr (kSwz == 32) {
+        if constexpr (kSwz == 0) {
+            // linear rows (1-D bulk copies): a thread's 32 bytes sit at 32r, so a quarter-warp's first loads
+            // would hit each 16-byte bank group twice; lanes with bit 2 set load their upper chunk first,
+            // which spreads every quarter-warp's 8 chunks over all 8 bank groups (conflict-free LDS.128)
+            const uint32_t rowa = row_base + rr * (4u * W);
+            const int4 A = ptx::lds128(rowa + g.off0);
+            const int4 B = ptx::lds128(rowa + g.off1);
+            q0 = g.swap ? B : A;
+            q1 = g.swap ? A : B;
+        } else if constexpr (kSwz == 32) {
             q0 = ptx::lds128(row_base + swz32(line, 0));
             q1 = ptx::lds128(row_base + swz32(line, 1));
         } else {
@@ -158,7 +171,9 @@ __device__ __forceinline__ void h_row(uint32_t row_base, uint32_t rr, const RepG
         const int32_t qp = q + p;
         int32_t dn = __shfl_down_sync(0xffffffffu, d, 1);
         int4 qn = q0;   // lane 31 / wrapping repetition: neighbour chunk from smem (predicated, no branch)
-        if constexpr (kSwz == 32)
+        if constexpr (kSwz == 0)
+            ptx::lds128_if(qn, row_base + rr * (4u * W) + g.offn, g.fix);
+        else if constexpr (kSwz == 32)
             ptx::lds128_if(qn, row_base + swz32(rr * segs + g.segn, 0), g.fix);
         else
             ptx::lds128_if(qn, row_base + swz(rr * segs + g.segn, g.offn), g.fix);
@@ -201,8 +216,9 @@ __device__ __forceinline__ void h_row(uint32_t row_base, uint32_t rr, const RepG
 // kR = repetitions of the H tiler per consumer thread: 1 for int32 (two LDS.128 already cover one repetition's
 // 8 columns); 1 or 2 for uint8 input, whose 16 bytes for two repetitions come in one LDS.128 and whose per-stage
 // bookkeeping (mbarrier wait/arrive, addressing) two repetitions then share (the host picks, fused.cu).
-// kSwz = the int32 smem layout: 128 (SWIZZLE_128B, W % 32 == 0) or 32 (SWIZZLE_32B, other W % 8 == 0);
-// unused (0) for uint8.  Tout = output element: int32, or int16 for 8-bit samples (outputs in [-5, 255]).
+// kSwz = the int32 smem layout: 128 (TMA tensor loads under SWIZZLE_128B, W % 32 == 0), 0 (1-D bulk copies,
+// linear rows, any W % 8 == 0; the default when W % 32 != 0) or 32 (TMA tensor loads of 32-byte lines under
+// SWIZZLE_32B, W % 8 == 0 and W <= 2048; an A/B alternative to 0); unused (0) for uint8.  Tout = output element: int32, or int16 for 8-bit samples (outputs in [-5, 255]).
 template <typename Tin, typename Tout, int kR, int kSwz, bool kChecksum, int kMaxThreads, int kMinBlocks>
 __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
     fused_tma_kernel(const __grid_constant__ CUtensorMap tmap, const FusedArgs a) {
@@ -230,7 +246,7 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
     if (tid >= NC) {
         // ------------------------------------------------ producer warp (TMA)
         if (tid == NC) {
-            if (kI32 || a.u8_tensor) ptx::prefetch_tensormap(&tmap);
+            if ((kI32 && kSwz != 0) || a.u8_tensor) ptx::prefetch_tensormap(&tmap);
             int s = 0;
             uint32_t ph = 0;
             for (int64_t k = 0, u = unit_of(a, 0); u < a.nunits; u = unit_of(a, ++k)) {
@@ -246,7 +262,11 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
                     ptx::mbar_wait_sleep(&empty[s], ph ^ 1u);   // suspended, not spinning, while the ring is full
                     ptx::mbar_arrive_expect_tx(&full[s], a.stage_bytes);
                     uint8_t* dst = stage_base + size_t(s) * a.stage_stride;
-                    if constexpr (kI32) {
+                    if constexpr (kI32 && kSwz == 0) {
+                        // linear layout: the triple is 12W contiguous bytes (16-byte multiple for W % 4 == 0)
+                        const uint8_t* src = static_cast<const uint8_t*>(a.X) + size_t(row0 + 3 * trip) * 4u * a.W;
+                        ptx::bulk_load(dst, src, a.stage_bytes, &full[s]);
+                    } else if constexpr (kI32) {
                         if (a.hint_loads)
                             ptx::tma_load_3d_hint(dst, &tmap, &full[s], 0, 0, int32_t(row0 + 3 * trip),
                                                   ptx::policy_evict_first());
@@ -276,7 +296,14 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
     const int rn = (r + kR == a.reps) ? 0 : r + kR;  // next thread's repetition (toroidal, Fig. 11 '% 1920')
     RepGeom g;
     g.fix = (lane == 31) || (r + 1 == a.reps);
-    if constexpr (kI32 && kSwz == 32) {
+    g.swap = false;
+    if constexpr (kI32 && kSwz == 0) {
+        g.seg = g.segn = 0;
+        g.swap = ((lane >> 2) & 1) != 0;   // r = tid, so r mod 8 = lane mod 8
+        g.off0 = 32u * uint32_t(r) + (g.swap ? 16u : 0u);
+        g.off1 = 32u * uint32_t(r) + (g.swap ? 0u : 16u);
+        g.offn = 32u * uint32_t(rn);
+    } else if constexpr (kI32 && kSwz == 32) {
         g.seg = uint32_t(r);   // one 32-byte line per repetition
         g.segn = uint32_t(rn);
         g.off0 = g.off1 = g.offn = 0;
@@ -549,7 +576,7 @@ __global__ void __launch_bounds__(256)
 using KernelFn = void (*)(const CUtensorMap, const FusedArgs);
 
 // Explicit instantiations live in fused_k_*.cu (compiled in parallel); these pick one.
-KernelFn tma_kernel_i32(bool checksum, bool swz32, int block, int cps);
+KernelFn tma_kernel_i32(bool checksum, int layout, int block, int cps);   // layout = kSwz (128, 32 or 0)
 KernelFn tma_kernel_u8(bool checksum, bool out16, int reps_per_thread, int block, int cps);
 
 template <typename Tin, typename Tout, int kR, int kSwz, bool kChecksum>

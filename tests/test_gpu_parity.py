@@ -97,16 +97,19 @@ def test_fused_launch_options(orc, opts):
     assert np.array_equal(np_u64(cs), cso)
 
 
-@pytest.mark.parametrize("shape", [(1, 1, 9, 8), (2, 3, 18, 40), (1, 3, 36, 1000), (2, 3, 27, 720), (1, 2, 18, 2040)])
-def test_swizzle32_shapes(orc, shape):
-    """int32, W % 32 != 0 (e.g. 720-wide SD frames): the TMA kernel with 32-byte lines under SWIZZLE_32B
-    ({8, W/8, 3} boxes, W <= 2048), against the oracle and the generic kernel, with and without checksums."""
+@pytest.mark.parametrize("shape", [(1, 1, 9, 8), (2, 3, 18, 40), (1, 3, 36, 1000), (2, 3, 27, 720), (1, 2, 18, 2040),
+                                   (1, 3, 18, 24), (2, 1, 27, 1448)])
+def test_unaligned_width_shapes(orc, shape):
+    """int32, W % 32 != 0 (e.g. 720-wide SD frames): the TMA kernel on linear rows (1-D bulk copies of the
+    row triple, lane-rotated LDS.128; the default), on 32-byte lines under SWIZZLE_32B (AOL_FLAG_I32_SWZ32 =
+    256, W <= 2048), against the oracle and the generic kernel, with and without checksums."""
     N, C, H, W = shape
     xh = synth.frames(5, 0, N, C, H, W, "signed")
     zo, cso = run_oracle(orc, xh)
     assert aol.downscale_frame_plan(N, C, H, W)["kernel"] == 1
     x = torch.from_numpy(xh).cuda()
-    for opts in (None, {"kernel": 1, "ctas_per_sm": 2, "bands_per_unit": 1}, {"kernel": 2}):
+    for opts in (None, {"kernel": 1, "ctas_per_sm": 2, "bands_per_unit": 1}, {"kernel": 1, "flags": 256},
+                 {"kernel": 1, "flags": 256, "ctas_per_sm": 3, "stages": 2}, {"kernel": 2}):
         z, cs = aol.downscale_frame(x, checksums=True, opts=opts)
         z2, _ = aol.downscale_frame(x, opts=opts)
         torch.cuda.synchronize()
@@ -115,19 +118,38 @@ def test_swizzle32_shapes(orc, shape):
         assert np.array_equal(np_u64(cs), cso), opts
 
 
-@pytest.mark.parametrize("shape", [(1, 1, 9, 2056), (1, 2, 18, 4008)])
-def test_generic_only_shapes(orc, shape):
-    """int32, W % 32 != 0 and W > 2048 (a box dimension holds <= 256 lines): the generic fused kernel."""
+@pytest.mark.parametrize("shape", [(2, 3, 36, 128), (1, 3, 27, 1920), (3, 1, 18, 352), (1, 1, 9, 32)])
+def test_linear_rows_forced(orc, shape):
+    """AOL_FLAG_I32_LINEAR (128): linear rows by 1-D bulk copies even when W % 32 == 0 (A/B against the
+    default SWIZZLE_128B tensor loads): same integers."""
+    N, C, H, W = shape
+    xh = synth.frames(6, 0, N, C, H, W, "uniform")
+    zo, cso = run_oracle(orc, xh)
+    x = torch.from_numpy(xh).cuda()
+    for opts in ({"kernel": 1, "flags": 128}, {"kernel": 1, "flags": 128, "ctas_per_sm": 2, "bands_per_unit": 2}):
+        z, cs = aol.downscale_frame(x, checksums=True, opts=opts)
+        torch.cuda.synchronize()
+        assert np.array_equal(z.cpu().numpy(), zo), opts
+        assert np.array_equal(np_u64(cs), cso), opts
+
+
+@pytest.mark.parametrize("shape", [(1, 1, 9, 2056), (1, 2, 18, 4008), (1, 1, 9, 7432)])
+def test_wide_unaligned_shapes(orc, shape):
+    """int32, W % 32 != 0 and W > 2048: linear rows (a TMA box dimension holds <= 256 lines, so the
+    SWIZZLE_32B layout cannot take these widths and falls back to the generic fused kernel)."""
     N, C, H, W = shape
     xh = synth.frames(5, 0, N, C, H, W, "signed")
     zo, cso = run_oracle(orc, xh)
-    assert aol.downscale_frame_plan(N, C, H, W)["kernel"] == 2
-    z, cs = aol.downscale_frame(torch.from_numpy(xh).cuda(), checksums=True)
-    torch.cuda.synchronize()
-    assert np.array_equal(z.cpu().numpy(), zo)
-    assert np.array_equal(np_u64(cs), cso)
+    assert aol.downscale_frame_plan(N, C, H, W)["kernel"] == 1
+    assert aol.downscale_frame_plan(N, C, H, W, opts={"flags": 256})["kernel"] == 2
+    x = torch.from_numpy(xh).cuda()
+    for opts in (None, {"flags": 256}):
+        z, cs = aol.downscale_frame(x, checksums=True, opts=opts)
+        torch.cuda.synchronize()
+        assert np.array_equal(z.cpu().numpy(), zo), opts
+        assert np.array_equal(np_u64(cs), cso), opts
     with pytest.raises(aol.AolError):
-        aol.downscale_frame(torch.from_numpy(xh).cuda(), opts={"kernel": 1})
+        aol.downscale_frame(x, opts={"kernel": 1, "flags": 256})
 
 
 @pytest.mark.parametrize("shape,kernel", [
