@@ -279,7 +279,7 @@ def test_frame_checksum_kernel(orc):
 
 # -------------------------------------------------------------- generic tilers
 
-@pytest.mark.parametrize("seed", range(200))
+@pytest.mark.parametrize("seed", range(1000))   # seeds 0..999
 def test_tiler_gather_scatter_vs_oracle(orc, seed):
     rng = np.random.default_rng(5000 + seed)
     d = bf.random_descriptor(rng)
@@ -307,6 +307,26 @@ def test_tiler_gather_scatter_vs_oracle(orc, seed):
         aol.tiler_scatter(gt, torch.from_numpy(Gs).cuda().reshape(G.shape), arr2, mode="fast")
         torch.cuda.synchronize()
         assert np.array_equal(arr2.cpu().numpy(), So)
+
+
+def test_tiler_d3_perf_instance_full_size(orc):
+    """SURVEY 8(d) d3 at the size tools/bench_configs.py times: array {64,1024,1024} int32 (256 MB), rep
+    {64,128,128}, pattern {8,8}, P = diag(1,8,8), F = [[0,0],[1,0],[0,1]] -- gather element by element
+    against the C oracle, and the FAST scatter of the tiles back into a zeroed array rebuilds the input
+    (the tiler is a bijection onto the array)."""
+    arr, rep, pat = [64, 1024, 1024], [64, 128, 128], [8, 8]
+    P, F = [[1, 0, 0], [0, 8, 0], [0, 0, 8]], [[0, 0], [1, 0], [0, 1]]
+    A = synth.frames(77, 0, 1, 64, 1024, 1024, "signed")[0]
+    ot = orc.make_tiler(arr, rep, pat, [0, 0, 0], P, F)
+    gt = aol.make_tiler(arr, rep, pat, [0, 0, 0], P, F)
+    Ad = torch.from_numpy(A).cuda()
+    G = aol.tiler_gather(gt, Ad)
+    torch.cuda.synchronize()
+    assert np.array_equal(G.cpu().numpy(), orc.gather(ot, A))
+    back = torch.zeros_like(Ad)
+    aol.tiler_scatter(gt, G, back, mode="fast")
+    torch.cuda.synchronize()
+    assert torch.equal(back, Ad)
 
 
 LINEAR_TILERS = [
@@ -509,6 +529,40 @@ def test_4k_batch(orc):
         _, cso = run_oracle(orc, synth.frames(1, n, 1, C, H, W, "uniform"))
         assert got[n] == cso[0], n
     del x, z
+    torch.cuda.empty_cache()
+
+
+def test_cif_2000_frames(orc):
+    """The paper's second workload (Section III): 2000 CIF frames 352x288 ->
+    132x128 in the launch tools/bench_configs.py times (4 CTAs/SM).  EVERY frame's checksum against the
+    oracle (one OpenMP oracle call over the whole batch), and frames {0, 999, 1999} element by element."""
+    N, C, H, W = 2000, 3, 288, 352
+    x = aol.synth_frames(4, 0, N, C, H, W, "uniform")
+    z, cs = aol.downscale_frame(x, checksums=True)
+    torch.cuda.synchronize()
+    zo, cso = orc.downscale_frame(x.cpu().numpy(), nthreads=16)
+    assert np.array_equal(np_u64(cs), cso)
+    for n in (0, 999, 1999):
+        assert np.array_equal(z[n].cpu().numpy(), zo[n]), n
+
+
+def test_u8_300_hd_frames_int16_out(orc):
+    """NEXT row f1 at bench size: 300 HD frames of 8-bit samples with int16 outputs (bench.py --dtype u8
+    --out-dtype i16, 3 CTAs/SM) and with int32 outputs: the checksums of both equal the int32-input path's
+    on the same integers, sampled frames element by element against the oracle."""
+    N, C, H, W = 300, 3, 1080, 1920
+    x8 = aol.synth_frames(0, 0, N, C, H, W, "uniform", dtype=torch.uint8)
+    z16, cs16 = aol.downscale_frame(x8, checksums=True, out_dtype=torch.int16)
+    z32, cs32 = aol.downscale_frame(x8, checksums=True)
+    torch.cuda.synchronize()
+    assert torch.equal(cs16.view(torch.int64), cs32.view(torch.int64))
+    assert torch.equal(z16.to(torch.int32), z32)
+    got = np_u64(cs16)
+    for n in (0, 150, 299):
+        zo, cso = run_oracle(orc, synth.frames(0, n, 1, C, H, W, "uniform"))
+        assert np.array_equal(z16[n:n + 1].cpu().numpy().astype(np.int32), zo), n
+        assert got[n] == cso[0], n
+    del x8, z16, z32
     torch.cuda.empty_cache()
 
 
