@@ -21,6 +21,8 @@
 
 #include <algorithm>
 #include <cstdint>
+#include <cstdlib>
+#include <cstring>
 
 #include "common.h"
 
@@ -251,6 +253,142 @@ __global__ void __launch_bounds__(256) tiler_linear32_kernel(const TilerDev td, 
     }
 }
 
+// ------------------------------------------------------------ wrapping tilers, 32-bit
+// Tilers whose pattern can leave the array (the paper's H/V input tilers wrap at the last repetition, Fig. 10
+// P:L681-687) with at most two wrapping array dims and all offsets < 2^31.  The flat offset is computed as if
+// nothing wrapped (one IMAD per combined dim, like the linear kernels) together with the raw coordinate of each
+// wrapping dim; the toroidal wrap is then one magic-number division per wrapping dim:
+//   (v mod s) * stride = v * stride - floor(v / s) * (s * stride).
+// Walked in tile order (tile side coalesced), all-32-bit, constants staged in shared memory.
+struct Wrap32Dev {
+    int32_t nd, nw;                                    // combined dims, wrapping array dims (0..2)
+    int32_t ext[2 * AOL_MAX_RANK], lin[2 * AOL_MAX_RANK];
+    uint32_t mul[2 * AOL_MAX_RANK], shift[2 * AOL_MAX_RANK];
+    int32_t wc[2][2 * AOL_MAX_RANK];                   // coefficient of combined dim d in wrapping dim k
+    int32_t worg[2], wext[2], wstep[2];                // origin, extent, extent * array stride
+    uint32_t wmul[2], wshift[2];
+    int32_t base, total;
+};
+
+template <int ES, int MODE>
+__global__ void __launch_bounds__(256) tiler_wrap32_kernel(const Wrap32Dev wd, const void* __restrict__ src,
+                                                           void* __restrict__ dst, unsigned long long* __restrict__ ws) {
+    using T = typename Elem<ES>::T;
+    __shared__ int4 pk[kND];   // {extent, magic multiplier, shift, flat-offset coefficient}
+    __shared__ int2 pw[kND];   // coefficients in the two wrapping dims
+    if (threadIdx.x < wd.nd) {
+        const int d = threadIdx.x;
+        pk[d] = make_int4(wd.ext[d], int32_t(wd.mul[d]), int32_t(wd.shift[d]), wd.lin[d]);
+        pw[d] = make_int2(wd.wc[0][d], wd.wc[1][d]);
+    }
+    __syncthreads();
+    const int32_t n_el = wd.total;
+    const int32_t stride = int32_t(gridDim.x * blockDim.x);
+    constexpr int kU = (MODE <= 1) ? 2 : 1;
+    const int32_t warp_first = int32_t((blockIdx.x * blockDim.x + (threadIdx.x & ~31u)) * kU + (threadIdx.x & 31u));
+    for (int32_t v0 = warp_first; v0 < n_el; v0 += kU * stride) {
+        int32_t off[kU], g[kU];
+#pragma unroll
+        for (int u = 0; u < kU; ++u) {
+            g[u] = v0 + 32 * u;
+            uint32_t n = g[u] < n_el ? uint32_t(g[u]) : 0u;
+            int32_t o = wd.base, w0 = wd.worg[0], w1 = wd.worg[1];
+#pragma unroll 1
+            for (int d = wd.nd - 1; d >= 0; --d) {
+                const int4 p = pk[d];
+                const int2 c = pw[d];
+                const uint32_t q = (__umulhi(n, uint32_t(p.y)) + n) >> p.z;
+                const int32_t i = int32_t(n - q * uint32_t(p.x));
+                n = q;
+                o += p.w * i;
+                w0 += c.x * i;
+                w1 += c.y * i;
+            }
+            if (wd.nw > 0) o -= int32_t((__umulhi(uint32_t(w0), wd.wmul[0]) + uint32_t(w0)) >> wd.wshift[0]) * wd.wstep[0];
+            if (wd.nw > 1) o -= int32_t((__umulhi(uint32_t(w1), wd.wmul[1]) + uint32_t(w1)) >> wd.wshift[1]) * wd.wstep[1];
+            off[u] = o;
+        }
+        if (MODE == 0) {   // gather: tiles[g] = array[off]
+            T val[kU];
+#pragma unroll
+            for (int u = 0; u < kU; ++u)
+                if (g[u] < n_el) val[u] = static_cast<const T*>(src)[off[u]];
+#pragma unroll
+            for (int u = 0; u < kU; ++u)
+                if (g[u] < n_el) static_cast<T*>(dst)[g[u]] = val[u];
+        } else if (MODE == 1) {   // FAST scatter: array[off] = tiles[g]
+            T val[kU];
+#pragma unroll
+            for (int u = 0; u < kU; ++u)
+                if (g[u] < n_el) val[u] = static_cast<const T*>(src)[g[u]];
+#pragma unroll
+            for (int u = 0; u < kU; ++u)
+                if (g[u] < n_el) static_cast<T*>(dst)[off[u]] = val[u];
+        } else if (MODE == 2) {   // SEQUENTIAL claim: the last (r, i) in row-major order wins
+            if (g[0] < n_el) atomicMax(ws + off[0], (unsigned long long)g[0] + 1ull);
+        } else {                  // SEQUENTIAL write
+            if (g[0] < n_el && ws[off[0]] == (unsigned long long)g[0] + 1ull)
+                static_cast<T*>(dst)[off[0]] = static_cast<const T*>(src)[g[0]];
+        }
+    }
+}
+
+// Fill *wd for a non-linear tiler if it qualifies (<= 2 wrapping dims, every unwrapped offset < 2^31).
+bool make_wrap32(const TilerDev& td, Wrap32Dev* wd) {
+    if (td.linear || !td.fast32 || td.array_elems >= (int64_t(1) << 31)) return false;
+    std::memset(wd, 0, sizeof *wd);
+    int wa[2], nw = 0;
+    for (int a = 0; a < td.ra; ++a)
+        if (!((td.nowrap_mask >> a) & 1)) {
+            if (nw == 2) return false;
+            wa[nw++] = a;
+        }
+    // the largest unwrapped flat offset: sum over array dims of (max raw coordinate) * stride
+    __int128 bound = 0;
+    for (int a = 0; a < td.ra; ++a) {
+        __int128 mx = td.org[a];
+        for (int d = 0; d < td.nd; ++d) mx += __int128(td.coef[a][d]) * (td.ext[d] - 1);
+        bound += mx * td.astride[a];
+    }
+    if (bound >= (__int128(1) << 31)) return false;
+    wd->nd = td.nd;
+    wd->nw = nw;
+    wd->total = int32_t(td.total);
+    int64_t base = 0;
+    for (int a = 0; a < td.ra; ++a) base += td.org[a] * td.astride[a];
+    wd->base = int32_t(base);
+    for (int d = 0; d < td.nd; ++d) {
+        int64_t l = 0;
+        for (int a = 0; a < td.ra; ++a) l += td.coef[a][d] * td.astride[a];
+        wd->ext[d] = int32_t(td.ext[d]);
+        wd->lin[d] = int32_t(l);
+        wd->mul[d] = td.fd_mul[d];
+        wd->shift[d] = td.fd_shift[d];
+        for (int k = 0; k < nw; ++k) wd->wc[k][d] = int32_t(td.coef[wa[k]][d]);
+    }
+    for (int k = 0; k < nw; ++k) {
+        const int a = wa[k];
+        const int64_t sa = td.ashape[a];
+        wd->worg[k] = int32_t(td.org[a]);
+        wd->wext[k] = int32_t(sa);
+        wd->wstep[k] = int32_t(sa * td.astride[a]);
+        uint32_t sh = 0;   // floor(v / s) == (umulhi(v, mul) + v) >> sh for v, s < 2^31
+        while (sh < 32 && (uint64_t(1) << sh) < uint64_t(sa)) ++sh;
+        wd->wmul[k] = uint32_t(((uint64_t(1) << 32) * ((uint64_t(1) << sh) - uint64_t(sa))) / uint64_t(sa) + 1);
+        wd->wshift[k] = sh;
+    }
+    return true;
+}
+
+// AOL_TILER_WRAP32=0 keeps wrapping tilers on the 64-bit general kernel (A/B measurements only).
+bool tiler_wrap32_enabled() {
+    static const bool v = [] {
+        const char* e = std::getenv("AOL_TILER_WRAP32");
+        return !(e && e[0] == '0');
+    }();
+    return v;
+}
+
 int grid_for(int64_t n, int num_sms) {
     return int(std::max<int64_t>(1, std::min<int64_t>((n + 255) / 256, int64_t(num_sms) * 32)));
 }
@@ -268,6 +406,18 @@ aol_status_t launch_v(const TilerDev& td, const void* src, void* dst, unsigned l
         AOL_LAUNCH_CHECK("tiler_linear32_kernel");
         return AOL_OK;
     }
+    if constexpr (V == 1) {
+        Wrap32Dev wd;
+        if (!lin && tiler_wrap32_enabled() && make_wrap32(td, &wd)) {
+            DeviceInfo dev;
+            aol_status_t st = device_info(&dev);
+            if (st != AOL_OK) return st;
+            const int gw = int(std::max<int64_t>(1, std::min<int64_t>((td.total + 255) / 256, int64_t(dev.num_sms) * 128)));
+            tiler_wrap32_kernel<ES, MODE><<<gw, 256, 0, s>>>(wd, src, dst, ws);
+            AOL_LAUNCH_CHECK("tiler_wrap32_kernel");
+            return AOL_OK;
+        }
+    }
     if (fast && lin)
         tiler_kernel<ES, V, true, true, MODE><<<grid, 256, 0, s>>>(td, src, dst, ws);
     else if (fast)
@@ -284,12 +434,27 @@ template <int ES, int MODE>
 aol_status_t launch_es(const TilerDev& td, int vec, const void* src, void* dst, unsigned long long* ws,
                        int num_sms, cudaStream_t s) {
     const int grid = grid_for(td.total / vec, num_sms);
-    // vector width in elements: 16 / ES when the host proved contiguity + alignment, else 1
-    if (vec > 1 && ES * vec == 16) {
-        if constexpr (ES == 1) return launch_v<1, 16, MODE>(td, src, dst, ws, grid, s);
-        if constexpr (ES == 2) return launch_v<2, 8, MODE>(td, src, dst, ws, grid, s);
-        if constexpr (ES == 4) return launch_v<4, 4, MODE>(td, src, dst, ws, grid, s);
-        if constexpr (ES == 8) return launch_v<8, 2, MODE>(td, src, dst, ws, grid, s);
+    // vector width in elements (16, 8, 4 or 2 bytes) when the host proved contiguity + alignment, else 1
+    if (vec > 1) {
+        const int vb = ES * vec;
+        if constexpr (ES == 1) {
+            if (vb == 16) return launch_v<1, 16, MODE>(td, src, dst, ws, grid, s);
+            if (vb == 8) return launch_v<1, 8, MODE>(td, src, dst, ws, grid, s);
+            if (vb == 4) return launch_v<1, 4, MODE>(td, src, dst, ws, grid, s);
+            if (vb == 2) return launch_v<1, 2, MODE>(td, src, dst, ws, grid, s);
+        }
+        if constexpr (ES == 2) {
+            if (vb == 16) return launch_v<2, 8, MODE>(td, src, dst, ws, grid, s);
+            if (vb == 8) return launch_v<2, 4, MODE>(td, src, dst, ws, grid, s);
+            if (vb == 4) return launch_v<2, 2, MODE>(td, src, dst, ws, grid, s);
+        }
+        if constexpr (ES == 4) {
+            if (vb == 16) return launch_v<4, 4, MODE>(td, src, dst, ws, grid, s);
+            if (vb == 8) return launch_v<4, 2, MODE>(td, src, dst, ws, grid, s);
+        }
+        if constexpr (ES == 8) {
+            if (vb == 16) return launch_v<8, 2, MODE>(td, src, dst, ws, grid, s);
+        }
     }
     return launch_v<ES, 1, MODE>(td, src, dst, ws, grid_for(td.total, num_sms), s);
 }
@@ -306,17 +471,20 @@ aol_status_t launch_mode(const TilerDev& td, int elsize, int vec, const void* sr
     return fail(AOL_E_DTYPE, "element size must be 1, 2, 4 or 8 bytes");
 }
 
-// Largest usable vector (elements): the permuted innermost dim is the natural last dim, unit-stride on
-// both sides; every other stride, the origin and the pointers keep V-element alignment.
+// Largest usable vector (elements; 16, 8, 4 or 2 bytes): the permuted innermost dim is the natural last dim,
+// unit-stride on both sides; every other stride, the origin and the pointers keep V-element alignment.
 int vector_width(const TilerDev& td, int elsize, const void* p_array, const void* p_tiles) {
-    const int v = 16 / elsize;
-    if (!td.linear || td.nd == 0 || v <= 1) return 1;
+    if (!td.linear || td.nd == 0) return 1;
     const int last = td.nd - 1;
-    if (td.p_lin[last] != 1 || td.p_gst[last] != 1 || td.p_ext[last] % v != 0 || td.base % v != 0) return 1;
-    for (int d = 0; d < last; ++d)
-        if (td.p_lin[d] % v != 0 || td.p_gst[d] % v != 0) return 1;
-    if ((reinterpret_cast<uintptr_t>(p_array) | reinterpret_cast<uintptr_t>(p_tiles)) % 16) return 1;
-    return v;
+    if (td.p_lin[last] != 1 || td.p_gst[last] != 1) return 1;
+    const uintptr_t ptrs = reinterpret_cast<uintptr_t>(p_array) | reinterpret_cast<uintptr_t>(p_tiles);
+    for (int vb = 16; vb > elsize; vb /= 2) {
+        const int v = vb / elsize;
+        bool ok = td.p_ext[last] % v == 0 && td.base % v == 0 && ptrs % vb == 0;
+        for (int d = 0; d < last && ok; ++d) ok = td.p_lin[d] % v == 0 && td.p_gst[d] % v == 0;
+        if (ok) return v;
+    }
+    return 1;
 }
 
 }  // namespace
