@@ -528,11 +528,21 @@ aol_status_t aol_downscale_frame_host(const void* h_in, aol_dtype_t in_dtype, in
     st = plan_fused(in_dtype, AOL_I32, d_in[0], d_out[0], chunk_frames, channels, H, W, nullptr, &plan);
     if (st != AOL_OK) return st;
 
-    cudaEvent_t ev_in[2], ev_comp[2], ev_out[2];
+    cudaEvent_t ev_in[2] = {}, ev_comp[2] = {}, ev_out[2] = {};
+    auto destroy_events = [&] {
+        for (int b = 0; b < 2; ++b)
+            for (cudaEvent_t ev : {ev_in[b], ev_comp[b], ev_out[b]})
+                if (ev) cudaEventDestroy(ev);
+    };
     for (int b = 0; b < 2; ++b) {
-        AOL_CUDA_TRY(cudaEventCreateWithFlags(&ev_in[b], cudaEventDisableTiming));
-        AOL_CUDA_TRY(cudaEventCreateWithFlags(&ev_comp[b], cudaEventDisableTiming));
-        AOL_CUDA_TRY(cudaEventCreateWithFlags(&ev_out[b], cudaEventDisableTiming));
+        cudaError_t ce = cudaEventCreateWithFlags(&ev_in[b], cudaEventDisableTiming);
+        if (ce == cudaSuccess) ce = cudaEventCreateWithFlags(&ev_comp[b], cudaEventDisableTiming);
+        if (ce == cudaSuccess) ce = cudaEventCreateWithFlags(&ev_out[b], cudaEventDisableTiming);
+        if (ce != cudaSuccess) {
+            destroy_events();
+            set_error("cudaEventCreate failed: %s", cudaGetErrorString(ce));
+            return AOL_E_CUDA;
+        }
     }
     aol_status_t result = AOL_OK;
     const uint8_t* hin = static_cast<const uint8_t*>(h_in);
@@ -576,11 +586,7 @@ aol_status_t aol_downscale_frame_host(const void* h_in, aol_dtype_t in_dtype, in
     cudaError_t e1 = cudaStreamSynchronize(s_d2h);
     cudaError_t e2 = cudaStreamSynchronize(s_compute);
     cudaError_t e3 = cudaStreamSynchronize(s_h2d);
-    for (int b = 0; b < 2; ++b) {
-        cudaEventDestroy(ev_in[b]);
-        cudaEventDestroy(ev_comp[b]);
-        cudaEventDestroy(ev_out[b]);
-    }
+    destroy_events();
     if (result == AOL_OK) {
         for (cudaError_t e : {e1, e2, e3})
             if (e != cudaSuccess) {

@@ -6,6 +6,7 @@
 #include <algorithm>
 #include <cstdint>
 #include <cstring>
+#include <vector>
 
 #include "common.h"
 #include "fused_kernel.cuh"
@@ -198,16 +199,30 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void*
         const int64_t max_ctas = int64_t(dev.num_sms) * cps;
         int nb = o.bands_per_unit;
         if (nb <= 0) {
-            // minimise (waves of units) x (triples per unit); prefer larger units on ties
-            int64_t best_cost = INT64_MAX;
-            for (int cand = 1; cand <= std::min(nbands, 40); ++cand) {
-                const int64_t upp = (nbands + cand - 1) / cand;
-                const int64_t units = planes * upp;
+            // Cost of a candidate: (units the busiest CTA runs) x (row triples per unit + a fixed per-unit cost in
+            // triple-equivalents).  int32 (HBM-bound): no fixed cost, and the SMALLEST unit within 2 % of the
+            // cheapest wins (a shorter last unit = a shorter tail; HD 1.240 ms at 10-12 bands vs 1.248 at 15, 4K
+            // 1.083 at 12 vs 1.089 at 24).  uint8 (issue-bound): the per-unit epilogue (checksum reduction,
+            // barriers) costs ~2 triples of a 1920-wide frame, inversely proportional to the row width, and the
+            // cheapest (largest on ties) wins (HD 0.479 ms at 20 bands vs 0.497 at 12, CIF 0.289 at 32 vs 0.310
+            // at 8; profiles/r01_nb_sweep.jsonl).
+            // (int16 outputs run 3 CTAs/SM: the epilogue weighs ~1.5x more; HD 0.421 ms at 20 vs 0.425 at 15)
+            const double ovh = in_dtype == AOL_U8 ? (out_es == 2 ? 5760.0 : 3840.0) / double(W) : 0.0;
+            const int max_nb = std::min(nbands, 120);
+            std::vector<double> cost(size_t(max_nb) + 1, 0.0);
+            double best = 1e300;
+            for (int cand = 1; cand <= max_nb; ++cand) {
+                const int64_t units = planes * ((nbands + cand - 1) / cand);
                 const int64_t waves = (units + max_ctas - 1) / max_ctas;
-                const int64_t cost = waves * (3 * cand + 1);
-                if (cost <= best_cost) {
-                    best_cost = cost;
-                    nb = cand;
+                cost[size_t(cand)] = double(waves) * (3.0 * cand + 1.0 + ovh);
+                best = std::min(best, cost[size_t(cand)]);
+            }
+            for (int cand = 1; cand <= max_nb; ++cand) {
+                if (in_dtype == AOL_U8) {
+                    if (cost[size_t(cand)] <= best) nb = cand;   // largest of the cheapest
+                } else if (cost[size_t(cand)] <= 1.02 * best) {
+                    nb = cand;                                   // smallest within 2 %
+                    break;
                 }
             }
         }

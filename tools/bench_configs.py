@@ -159,7 +159,26 @@ def main():
               "gather_GBps": nb / (tg / 1e3) / 1e9, "scatter_fast_ms": ts, "scatter_fast_GBps": nb / (ts / 1e3) / 1e9,
               "scatter_seq_ms": tq, "gather_frac": nb / (tg / 1e3) / 1e9 / peak(),
               "check_gather_is_blocking": bool(torch.equal(G[1, 2, 3], A[1, 16:24, 24:32]))})
+        # the same blocking with origin (0, -3, 5): tiles wrap toroidally in both image dims (BASELINE configs[2]
+        # "incl. modulo wrap-around"); and the paper's H input tiler (Fig. 10) over 64 HD planes
+        tw = aol.make_tiler([64, 1024, 1024], [64, 128, 128], [8, 8], [0, -3, 5],
+                            [[1, 0, 0], [0, 8, 0], [0, 0, 8]], [[0, 0], [1, 0], [0, 1]])
+        twg, _ = timed(lambda: aol.tiler_gather(tw, A, out=G))
+        tws, _ = timed(lambda: aol.tiler_scatter(tw, G, B, mode="fast"))
+        emit({"config": "d3 generic tiler, wrapping in both dims (origin (0,-3,5))", "gather_ms": twg,
+              "gather_GBps": nb / (twg / 1e3) / 1e9, "scatter_fast_ms": tws, "scatter_fast_GBps": nb / (tws / 1e3) / 1e9,
+              "check_wrap": bool(torch.equal(G[0, 0, 0, 0], A[0, 1021, 5:13])), "roundtrip_ok": bool(torch.equal(A, B))})
         del A, G, B
+        torch.cuda.empty_cache()
+        X = aol.synth_frames(0, 0, 64, 1, 1080, 1920).reshape(64, 1080, 1920)
+        th = aol.make_tiler([64, 1080, 1920], [64, 1080, 240], [11], [0, 0, 0],
+                            [[1, 0, 0], [0, 1, 0], [0, 0, 8]], [[0], [0], [1]])
+        GH = torch.empty((64, 1080, 240, 11), dtype=torch.int32, device="cuda")
+        thg, _ = timed(lambda: aol.tiler_gather(th, X, out=GH))
+        emit({"config": "H_IN tiler (Fig. 10) gather over 64 HD planes", "gather_ms": thg,
+              "gather_GBps": (X.numel() + GH.numel()) * 4 / (thg / 1e3) / 1e9,
+              "check_wrap": bool(torch.equal(GH[0, 0, 239], torch.cat([X[0, 0, 1912:1920], X[0, 0, 0:3]])))})
+        del X, GH
         torch.cuda.empty_cache()
     if want("f3"):
         # the paper's generic-vs-non-generic experiment on B200: run-time descriptors,
