@@ -18,7 +18,8 @@
 __device__ __forceinline__ uint32_t sa(const void* p) { return uint32_t(__cvta_generic_to_shared(p)); }
 
 __global__ void __launch_bounds__(32) stream_kernel(const uint8_t* __restrict__ src, uint8_t* __restrict__ dst,
-                                                    size_t read_bytes, size_t chunk, int stages, int wpm) {
+                                                    size_t read_bytes, size_t chunk, int stages, int wpm,
+                                                    int inter) {
     extern __shared__ __align__(1024) uint8_t smem[];
     uint64_t* bar = reinterpret_cast<uint64_t*>(smem + size_t(stages) * chunk);
     if (threadIdx.x != 0) return;
@@ -27,9 +28,15 @@ __global__ void __launch_bounds__(32) stream_kernel(const uint8_t* __restrict__ 
     asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
     const size_t nchunks = read_bytes / chunk;
     const size_t per = (nchunks + gridDim.x - 1) / gridDim.x;
-    const size_t c0 = blockIdx.x * per, c1 = c0 + per < nchunks ? c0 + per : nchunks;
+    const size_t b0 = blockIdx.x * per, b1 = b0 + per < nchunks ? b0 + per : nchunks;
+    // inter = 0: a contiguous block of chunks per CTA; 1: chunk k of this CTA is blockIdx.x + k * gridDim.x
+    // (round-robin, like the fused kernel's work units: concurrently running CTAs read adjacent chunks)
+    const size_t c0 = 0;
+    const size_t c1 = inter ? (blockIdx.x < nchunks ? (nchunks - blockIdx.x + gridDim.x - 1) / gridDim.x : 0)
+                            : (b1 > b0 ? b1 - b0 : 0);
+    auto at = [&](size_t k) { return inter ? blockIdx.x + k * gridDim.x : b0 + k; };
+    const uint32_t wb = uint32_t(chunk * wpm / 1000) & ~15u;
     uint32_t phase[64] = {0};
-    size_t wr = wpm ? (c0 * chunk * wpm / 1000) & ~size_t(15) : 0;   // this CTA slice of the write buffer (16 B aligned)
     size_t issued = c0;
     // prologue: fill the ring
     for (int s = 0; s < stages && issued < c1; ++s, ++issued) {
@@ -37,7 +44,7 @@ __global__ void __launch_bounds__(32) stream_kernel(const uint8_t* __restrict__ 
                      : "memory");
         asm volatile("cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];" ::"r"(
                          sa(smem + size_t(s) * chunk)),
-                     "l"(src + issued * chunk), "r"(uint32_t(chunk)), "r"(sa(&bar[s]))
+                     "l"(src + at(issued) * chunk), "r"(uint32_t(chunk)), "r"(sa(&bar[s]))
                      : "memory");
     }
     int s = 0;
@@ -50,13 +57,11 @@ __global__ void __launch_bounds__(32) stream_kernel(const uint8_t* __restrict__ 
                          : "memory");
         phase[s] ^= 1u;
         if (wpm > 0) {   // write chunk*wpm/1000 bytes of what just arrived
-            const uint32_t wb = uint32_t(chunk * wpm / 1000) & ~15u;
-            asm volatile("cp.async.bulk.global.shared::cta.bulk_group [%0], [%1], %2;" ::"l"(dst + wr),
+            asm volatile("cp.async.bulk.global.shared::cta.bulk_group [%0], [%1], %2;" ::"l"(dst + at(c) * wb),
                          "r"(sa(smem + size_t(s) * chunk)), "r"(wb)
                          : "memory");
             asm volatile("cp.async.bulk.commit_group;" ::: "memory");
             asm volatile("cp.async.bulk.wait_group.read 0;" ::: "memory");
-            wr += wb;
         }
         if (issued < c1) {
             asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(sa(&bar[s])),
@@ -65,7 +70,7 @@ __global__ void __launch_bounds__(32) stream_kernel(const uint8_t* __restrict__ 
             asm volatile(
                 "cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];" ::"r"(
                     sa(smem + size_t(s) * chunk)),
-                "l"(src + issued * chunk), "r"(uint32_t(chunk)), "r"(sa(&bar[s]))
+                "l"(src + at(issued) * chunk), "r"(uint32_t(chunk)), "r"(sa(&bar[s]))
                 : "memory");
             ++issued;
         }
@@ -88,9 +93,17 @@ int main(int argc, char** argv) {
     cudaEvent_t a, b;
     cudaEventCreate(&a);
     cudaEventCreate(&b);
-    struct Cfg { size_t chunk; int stages, wpm, cps; };
+    struct Cfg { size_t chunk; int stages, wpm, cps, inter = 0; };
     std::vector<Cfg> cfgs;
-    if (!u8) {
+    if (argc > 1 && std::string(argv[1]) == "inter") {
+        // blocked vs round-robin chunk order, int32 mix (166) and read-only, around the fused kernel's point
+        for (int inter : {0, 1})
+            for (int wpm : {166, 0})
+                for (size_t chunk : {size_t(16384), size_t(23040)})
+                    for (int stages : {4, 5, 6})
+                        for (int cps : {1, 2})
+                            if (chunk * stages * cps + 1024 * cps <= 220 * 1024) cfgs.push_back({chunk, stages, wpm, cps, inter});
+    } else if (!u8) {
         for (int wpm : {166, 0})
             for (size_t chunk : {size_t(16384), size_t(23040), size_t(32768)})
                 for (int stages : {2, 4, 6, 8})
@@ -111,19 +124,19 @@ int main(int argc, char** argv) {
         const int smem = int(c.chunk * c.stages + 64 * 8);
         cudaFuncSetAttribute(stream_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
         const int grid = sms * c.cps;
-        for (int w = 0; w < 2; ++w) stream_kernel<<<grid, 32, smem>>>(src, dst, read_bytes, c.chunk, c.stages, c.wpm);
+        for (int w = 0; w < 2; ++w) stream_kernel<<<grid, 32, smem>>>(src, dst, read_bytes, c.chunk, c.stages, c.wpm, c.inter);
         cudaEventRecord(a);
         const int reps = 10;
-        for (int r = 0; r < reps; ++r) stream_kernel<<<grid, 32, smem>>>(src, dst, read_bytes, c.chunk, c.stages, c.wpm);
+        for (int r = 0; r < reps; ++r) stream_kernel<<<grid, 32, smem>>>(src, dst, read_bytes, c.chunk, c.stages, c.wpm, c.inter);
         cudaEventRecord(b);
         cudaEventSynchronize(b);
         float ms = 0;
         cudaEventElapsedTime(&ms, a, b);
         ms /= reps;
         const double bytes = double(read_bytes) + double(read_bytes) * c.wpm / 1000.0;
-        printf("{\"chunk\": %zu, \"stages\": %d, \"ctas_per_sm\": %d, \"write_permille\": %d, \"ms\": %.4f, "
-               "\"GBps\": %.1f, \"err\": \"%s\"}\n",
-               c.chunk, c.stages, c.cps, c.wpm, ms, bytes / (ms * 1e-3) / 1e9, cudaGetErrorString(cudaGetLastError()));
+        printf("{\"chunk\": %zu, \"stages\": %d, \"ctas_per_sm\": %d, \"write_permille\": %d, \"interleaved\": %d, "
+               "\"ms\": %.4f, \"GBps\": %.1f, \"err\": \"%s\"}\n",
+               c.chunk, c.stages, c.cps, c.wpm, c.inter, ms, bytes / (ms * 1e-3) / 1e9, cudaGetErrorString(cudaGetLastError()));
     }
     return 0;
 }
