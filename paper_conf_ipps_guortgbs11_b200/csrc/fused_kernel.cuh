@@ -377,8 +377,8 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
                     } else {   // int16 pairs packed into 32-bit stores (e0 even)
 #pragma unroll
                         for (int m = 0; m < kC; m += 2)
-                            ptx::sts32(ob + 2u * (e0 + m),
-                                       int32_t((uint32_t(z[k][m]) & 0xffffu) | (uint32_t(z[k][m + 1]) << 16)));
+                            ptx::sts32(ob + 2u * (e0 + m),   // low halves of both values: one PRMT
+                                       int32_t(__byte_perm(uint32_t(z[k][m]), uint32_t(z[k][m + 1]), 0x5410u)));
                     }
                 }
             }

@@ -27,7 +27,9 @@ def main():
     torch.cuda.set_device(0)
     ok = True
     # W = 1040: uint8 two-repetitions-per-thread path with a partly idle warp and 1-D bulk copies
-    shapes = [(2, 3, 27, 64), (1, 1, 9, 32), (1, 2, 18, 352), (2, 2, 18, 256), (1, 1, 18, 1040)]
+    # W = 40 / 1000: int32 rows with W % 32 != 0 (linear smem rows filled by 1-D bulk copies)
+    shapes = [(2, 3, 27, 64), (1, 1, 9, 32), (1, 2, 18, 352), (2, 2, 18, 256), (1, 1, 18, 1040), (1, 2, 18, 40),
+              (1, 1, 9, 1000)]
     if args.widths:
         shapes = [sh for sh in shapes if str(sh[3]) in args.widths.split(",")]
     for (N, C, H, W) in shapes:
@@ -72,6 +74,12 @@ def main():
     G2 = aol.tiler_gather(tw, A[:9, :10].contiguous())
     C2 = torch.zeros((9, 10), dtype=torch.int32, device="cuda")
     aol.tiler_scatter(tw, G2, C2, mode="sequential")
+    # a bijective blocking shifted to wrap in both dims (32-bit wrapping kernel): FAST scatter inverts the gather
+    ts = aol.make_tiler([16, 24], [2, 3], [8, 8], [-3, 5], [[8, 0], [0, 8]], [[1, 0], [0, 1]])
+    G3 = aol.tiler_gather(ts, A)
+    D = torch.zeros_like(A)
+    aol.tiler_scatter(ts, G3, D, mode="fast")
+    ok &= torch.equal(A, D)
     # generic run-time filters (register-pattern kernel: 128-bit contiguous path, wrapping path, stepping)
     P, H, W = 2, 18, 256
     x = aol.synth_frames(3, 0, 1, P, H, W, "uniform")[0]
