@@ -121,6 +121,9 @@ typedef struct {
                                           W % 32 == 0 (default there: TMA tensor loads, SWIZZLE_128B) */
 #define AOL_FLAG_I32_SWZ32 256         /* int32 input, W % 32 != 0, W <= 2048: TMA tensor loads of
                                           32-byte lines under SWIZZLE_32B (default: linear rows)     */
+#define AOL_FLAG_ROW_STAGES 512        /* int32 input: one row per TMA ring stage (default when a row
+                                          triple exceeds a third of the ring's bytes: W > 3271)        */
+#define AOL_FLAG_TRIPLE_STAGES 1024    /* int32 input: one row triple per ring stage for any W       */
 
 /* The launch configuration aol_downscale_frame_ex would use (for reports/tests). */
 typedef struct {

@@ -80,9 +80,18 @@ KernelFn pick(aol_dtype_t dt, int out_es, bool checksum, int kr, int64_t W, int 
                         : tma_kernel_i32(checksum, i32_layout(dt, W, flags), block, cps);
 }
 
-// Shared-memory geometry of the TMA ring: one stage = one row triple.
+// Rows per ring stage: a row triple, or (int32) one row when a triple would be coarser than a third of the
+// bytes the ring keeps in flight (4K: 46 KB triples vs 115 KB per SM), unless forced by a flag.
+int rows_per_stage(aol_dtype_t dt, int64_t W, int flags) {
+    if (dt != AOL_I32) return 3;
+    if (flags & AOL_FLAG_ROW_STAGES) return 1;
+    if (flags & AOL_FLAG_TRIPLE_STAGES) return 3;
+    return 12 * W > kInflightBytesPerSM / 3 ? 1 : 3;
+}
+
+// Shared-memory geometry of the TMA ring: one stage = one row triple (or one row, rows_per_stage).
 struct RingGeom {
-    uint32_t stage_bytes;   // 3 rows of the input
+    uint32_t stage_bytes;   // rows_per_stage rows of the input
     uint32_t stage_stride;  // rounded up: 1024 B (SWIZZLE_128B atom) for int32, 128 B for uint8
     uint32_t out_bytes;     // one band of output: 4 rows of Wo output elements
 };
@@ -91,7 +100,7 @@ RingGeom ring_geom(aol_dtype_t dt, int out_es, int64_t W, int flags) {
     // swizzled layouts need 1024-byte aligned stages (the swizzle atom); bulk copies 16 bytes (128 kept)
     const uint32_t es = dt == AOL_U8 ? 1u : 4u, align = i32_layout(dt, W, flags) > 0 ? 1024u : 128u;
     RingGeom g;
-    g.stage_bytes = uint32_t(3 * W) * es;
+    g.stage_bytes = uint32_t(rows_per_stage(dt, W, flags) * W) * es;
     g.stage_stride = (g.stage_bytes + align - 1) & ~(align - 1);
     g.out_bytes = uint32_t(4 * out_es * (3 * (W / 8)));
     return g;
@@ -113,7 +122,7 @@ aol_status_t encode_row_map(CUtensorMap* map, aol_dtype_t dt, const void* base, 
     const cuuint64_t inner = i32 ? (s32 ? 8 : 32) : 128, es = i32 ? 4 : 1;
     const cuuint64_t gdim[3] = {inner, cuuint64_t(W) / inner, cuuint64_t(rows)};
     const cuuint64_t gstride[2] = {inner * es, cuuint64_t(W) * es};
-    const cuuint32_t box[3] = {cuuint32_t(inner), cuuint32_t(W / int64_t(inner)), 3};
+    const cuuint32_t box[3] = {cuuint32_t(inner), cuuint32_t(W / int64_t(inner)), cuuint32_t(rows_per_stage(dt, W, flags))};
     const cuuint32_t estr[3] = {1, 1, 1};
     CUresult cr = encode(map, i32 ? CU_TENSOR_MAP_DATA_TYPE_INT32 : CU_TENSOR_MAP_DATA_TYPE_UINT8, 3,
                          const_cast<void*>(base), gdim, gstride, box, estr, CU_TENSOR_MAP_INTERLEAVE_NONE,
@@ -171,7 +180,10 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void*
             if (o.stages > 0) {
                 stages = std::min(stages, o.stages);
             } else {
-                const int target = (kInflightBytesPerSM / cps + int(geom.stage_stride) / 2) / int(geom.stage_stride);
+                // nearest whole number of stages to the in-flight target; one-row stages round down (4K: 7 rows =
+                // 1.065 ms, 8 = 1.070, 9 = 1.13-1.16: HBM efficiency falls off a cliff above ~120 KB per SM)
+                const int half = rows_per_stage(in_dtype, W, o.flags) == 1 ? 0 : int(geom.stage_stride) / 2;
+                const int target = (kInflightBytesPerSM / cps + half) / int(geom.stage_stride);
                 stages = std::min(stages, std::max(2, target));
             }
             int occ = 0;
@@ -287,6 +299,7 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
     }
     FusedArgs a;
     a.u8_tensor = u8_tensor ? 1 : 0;
+    a.rows_per_stage = rows_per_stage(in_dtype, W, plan.flags);
     a.Z = d_out;
     a.cs = d_cs;
     a.X = d_in;

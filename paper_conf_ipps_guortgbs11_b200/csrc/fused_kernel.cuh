@@ -105,6 +105,8 @@ struct FusedArgs {
     int32_t hint_stores;    // 1: bulk stores with L2 evict_first
     int32_t blocked_units;  // 1: contiguous block of units per CTA instead of round-robin
     int32_t u8_tensor;      // uint8 path: 1 = 3-D TMA tensor loads (W % 128 == 0), 0 = 1-D bulk copies
+    int32_t rows_per_stage; // int32 path: 3 (a stage holds a row triple) or 1 (one row per stage: finer ring
+                            // granularity for wide frames); always 3 for uint8
 };
 
 // Byte offset of 16-byte chunk `chunk` (0..7) of 128-byte line `line` under SWIZZLE_128B
@@ -259,6 +261,26 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
                 const int32_t halo = (3 * b1 == a.triples_per_plane) ? 0 : 3 * b1;
                 for (int32_t t = 0; t < ntrip; ++t) {
                     const int32_t trip = t == 0 ? halo : 3 * b0 + t - 1;
+                    if constexpr (kI32) {
+                        if (a.rows_per_stage == 1) {   // one row per stage, three stages per triple
+                            for (int32_t q = 0; q < 3; ++q) {
+                                ptx::mbar_wait_sleep(&empty[s], ph ^ 1u);
+                                ptx::mbar_arrive_expect_tx(&full[s], a.stage_bytes);
+                                uint8_t* dst = stage_base + size_t(s) * a.stage_stride;
+                                const int64_t row = row0 + 3 * trip + q;
+                                if constexpr (kSwz == 0)
+                                    ptx::bulk_load(dst, static_cast<const uint8_t*>(a.X) + size_t(row) * 4u * a.W,
+                                                   a.stage_bytes, &full[s]);
+                                else
+                                    ptx::tma_load_3d(dst, &tmap, &full[s], 0, 0, int32_t(row));
+                                if (++s == a.stages) {
+                                    s = 0;
+                                    ph ^= 1u;
+                                }
+                            }
+                            continue;
+                        }
+                    }
                     ptx::mbar_wait_sleep(&empty[s], ph ^ 1u);   // suspended, not spinning, while the ring is full
                     ptx::mbar_arrive_expect_tx(&full[s], a.stage_bytes);
                     uint8_t* dst = stage_base + size_t(s) * a.stage_stride;
@@ -409,6 +431,22 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
 
         // Wait for the next ring stage, run the H stage on its 3 rows (y[row][col]), release the stage.
         auto triple = [&](int32_t (&y)[3][kC]) {
+            if constexpr (kI32) {
+                if (a.rows_per_stage == 1) {   // three one-row stages
+#pragma unroll
+                    for (int rr = 0; rr < 3; ++rr) {
+                        ptx::mbar_wait_sleep(&full[s], ph);
+                        h_row<Tin, kR, kSwz>(stage_s32 + uint32_t(s) * a.stage_stride, 0u, g, segs, Wu, y[rr]);
+                        __syncwarp();
+                        if (lane == 0) ptx::mbar_arrive(&empty[s]);
+                        if (++s == a.stages) {
+                            s = 0;
+                            ph ^= 1u;
+                        }
+                    }
+                    return;
+                }
+            }
             ptx::mbar_wait_sleep(&full[s], ph);
             const uint32_t sb = stage_s32 + uint32_t(s) * a.stage_stride;   // 32-bit shared address
 #pragma unroll

@@ -118,6 +118,29 @@ def test_unaligned_width_shapes(orc, shape):
         assert np.array_equal(np_u64(cs), cso), opts
 
 
+@pytest.mark.parametrize("shape", [(2, 3, 36, 128), (1, 3, 27, 1920), (1, 2, 18, 3840), (2, 1, 27, 720),
+                                   (1, 1, 9, 4008)])
+def test_row_and_triple_stages(orc, shape):
+    """int32 ring stages of one row (AOL_FLAG_ROW_STAGES = 512; the default for W > 3271) and of one row
+    triple (AOL_FLAG_TRIPLE_STAGES = 1024), on both smem layouts (+ AOL_FLAG_I32_LINEAR = 128) and with small
+    rings: identical integers."""
+    N, C, H, W = shape
+    xh = synth.frames(8, 0, N, C, H, W, "signed")
+    zo, cso = run_oracle(orc, xh)
+    x = torch.from_numpy(xh).cuda()
+    for flags in (512, 1024, 512 | 128, 1024 | 128):
+        for extra in ({}, {"stages": 2, "bands_per_unit": 1}, {"ctas_per_sm": 2, "stages": 3}):
+            o = dict(extra, kernel=1, flags=flags)
+            try:
+                z, cs = aol.downscale_frame(x, checksums=True, opts=o)
+            except aol.AolError:
+                assert W > 3271 and flags & 1024   # a triple ring may not fit next to 2 CTAs of wide frames
+                continue
+            torch.cuda.synchronize()
+            assert np.array_equal(z.cpu().numpy(), zo), o
+            assert np.array_equal(np_u64(cs), cso), o
+
+
 @pytest.mark.parametrize("shape", [(2, 3, 36, 128), (1, 3, 27, 1920), (3, 1, 18, 352), (1, 1, 9, 32)])
 def test_linear_rows_forced(orc, shape):
     """AOL_FLAG_I32_LINEAR (128): linear rows by 1-D bulk copies even when W % 32 == 0 (A/B against the
@@ -595,14 +618,18 @@ def test_host_streamed_u8_and_ragged_chunks(orc, chunk):
 
 # -------------------------------------------------------------- edge cases
 
-@pytest.mark.parametrize("W,dtype,kernel", [(7680, torch.int32, 1), (7936, torch.int32, 2), (7936, torch.uint8, 1),
-                                            (8192, torch.uint8, 2), (16, torch.uint8, 1), (32, torch.int32, 1)])
+@pytest.mark.parametrize("W,dtype,kernel", [(7680, torch.int32, 1), (7936, torch.int32, 1), (7944, torch.int32, 2),
+                                            (7936, torch.uint8, 1), (8192, torch.uint8, 2), (16, torch.uint8, 1),
+                                            (32, torch.int32, 1), (7432, torch.int32, 1)])
 def test_width_limits(orc, W, dtype, kernel):
-    """Widest frames the TMA kernel takes and the first widths that fall back to the generic kernel: int32
-    needs two 3-row stages + one 4-row output band in 227 KB of smem (W <= 7680); uint8 is capped by
-    W/8 <= 992 consumer threads + 1 producer warp = 1024.  Also the narrowest TMA widths."""
+    """Widest frames the TMA kernel takes and the first widths that fall back to the generic kernel: both
+    dtypes are capped by W/8 <= 992 consumer threads + 1 producer warp = 1024 (wide int32 frames stream one
+    row per ring stage, so two stages + one 4-row output band fit in 227 KB of smem up to W = 7936).  Also
+    the narrowest TMA widths."""
     N, C, H = 1, 1, 18
     xh = synth.frames(61, 0, N, C, H, W, "uniform")
+    if dtype == torch.int32 and kernel == 1 and W > 3271:
+        assert aol.downscale_frame_plan(N, C, H, W)["stages"] >= 2
     zo, cso = run_oracle(orc, xh)
     x = torch.from_numpy(xh.astype(np.uint8) if dtype == torch.uint8 else xh).cuda()
     assert aol.downscale_frame_plan(N, C, H, W, dtype=dtype)["kernel"] == kernel
