@@ -380,6 +380,170 @@ bool make_wrap32(const TilerDev& td, Wrap32Dev* wd) {
     return true;
 }
 
+// Gather / FAST scatter of the same tilers in blocks: the tile index space (natural order, tile side
+// contiguous) splits into INNER dims (the innermost ones, the outermost of them possibly in chunks) whose
+// product fills a block of <= kWTab elements, and OUTER dims enumerating the blocks.  Every block shares the
+// inner parts of the unwrapped flat offset and of the wrapping coordinates, so each CTA tabulates them once in
+// shared memory; an element then costs one LDS.128, three adds and the wrap fix-up instead of a digit-by-digit
+// decomposition (the per-element kernel above is issue/latency-bound on exactly that).
+constexpr int kWTab = 2048;   // 32 KB of int4 per CTA: 1024 entries 2.84 / 4096 2.61 / 2048 3.29 TB/s (wrapping d3)
+
+struct WrapTabDev {
+    int32_t n_in, n_out, nw;
+    int32_t in_ext[2 * AOL_MAX_RANK], in_lin[2 * AOL_MAX_RANK], in_w0[2 * AOL_MAX_RANK], in_w1[2 * AOL_MAX_RANK];
+    uint32_t in_mul[2 * AOL_MAX_RANK], in_shift[2 * AOL_MAX_RANK];
+    int32_t out_ext[2 * AOL_MAX_RANK + 1], out_lin[2 * AOL_MAX_RANK + 1], out_w0[2 * AOL_MAX_RANK + 1],
+        out_w1[2 * AOL_MAX_RANK + 1], out_g[2 * AOL_MAX_RANK + 1];
+    uint32_t out_mul[2 * AOL_MAX_RANK + 1], out_shift[2 * AOL_MAX_RANK + 1];
+    int32_t chunk_ext, chunk_len, inner, inner_tail, nblocks;
+    int32_t base, worg0, worg1, wext0, wext1, wstep0, wstep1;
+    uint32_t wmul0, wshift0, wmul1, wshift1;
+};
+
+template <int ES, int MODE>
+__global__ void __launch_bounds__(256) tiler_wraptab_kernel(const WrapTabDev wt, const void* __restrict__ src,
+                                                            void* __restrict__ dst) {
+    using T = typename Elem<ES>::T;
+    constexpr int kPer = kWTab / 256;
+    __shared__ int4 tab[kWTab];   // {flat offset, wrapping coordinate 0, wrapping coordinate 1} of the inner index
+    for (int e = threadIdx.x; e < wt.inner; e += 256) {
+        uint32_t n = uint32_t(e);
+        int32_t o = 0, w0 = 0, w1 = 0;
+        for (int d = wt.n_in - 1; d >= 0; --d) {
+            const uint32_t q = (__umulhi(n, wt.in_mul[d]) + n) >> wt.in_shift[d];
+            const int32_t i = int32_t(n - q * uint32_t(wt.in_ext[d]));
+            n = q;
+            o += wt.in_lin[d] * i;
+            w0 += wt.in_w0[d] * i;
+            w1 += wt.in_w1[d] * i;
+        }
+        tab[e] = make_int4(o, w0, w1, 0);
+    }
+    __syncthreads();
+    for (int32_t blk = blockIdx.x; blk < wt.nblocks; blk += gridDim.x) {
+        uint32_t n = uint32_t(blk);
+        int32_t bo = wt.base, b0 = wt.worg0, b1 = wt.worg1, bg = 0, count = wt.inner;
+        for (int d = wt.n_out - 1; d >= 0; --d) {
+            const uint32_t q = (__umulhi(n, wt.out_mul[d]) + n) >> wt.out_shift[d];
+            const int32_t i = int32_t(n - q * uint32_t(wt.out_ext[d]));
+            n = q;
+            bo += wt.out_lin[d] * i;
+            b0 += wt.out_w0[d] * i;
+            b1 += wt.out_w1[d] * i;
+            bg += wt.out_g[d] * i;
+            if (d == wt.n_out - 1)   // the chunk index: a partial last chunk holds fewer elements
+                count = min(wt.chunk_len, wt.chunk_ext - i * wt.chunk_len) * wt.inner_tail;
+        }
+        int32_t off[kPer];
+        T val[kPer];
+#pragma unroll
+        for (int k = 0; k < kPer; ++k) {
+            const int e = threadIdx.x + 256 * k;
+            const int4 t = tab[e < count ? e : 0];
+            int32_t o = bo + t.x;
+            const uint32_t w0 = uint32_t(b0 + t.y), w1 = uint32_t(b1 + t.z);
+            if (wt.nw > 0) o -= int32_t((__umulhi(w0, wt.wmul0) + w0) >> wt.wshift0) * wt.wstep0;
+            if (wt.nw > 1) o -= int32_t((__umulhi(w1, wt.wmul1) + w1) >> wt.wshift1) * wt.wstep1;
+            off[k] = o;
+        }
+#pragma unroll
+        for (int k = 0; k < kPer; ++k) {
+            const int e = threadIdx.x + 256 * k;
+            if (e < count) val[k] = MODE == 0 ? static_cast<const T*>(src)[off[k]] : static_cast<const T*>(src)[bg + e];
+        }
+#pragma unroll
+        for (int k = 0; k < kPer; ++k) {
+            const int e = threadIdx.x + 256 * k;
+            if (e < count) {
+                if (MODE == 0)
+                    static_cast<T*>(dst)[bg + e] = val[k];
+                else
+                    static_cast<T*>(dst)[off[k]] = val[k];
+            }
+        }
+    }
+}
+
+void magic32(int64_t ext, uint32_t* mul, uint32_t* shift) {
+    // n / ext == (umulhi(n, mul) + n) >> shift for n, ext < 2^31
+    uint32_t sh = 0;
+    while (sh < 32 && (uint64_t(1) << sh) < uint64_t(ext)) ++sh;
+    *mul = uint32_t(((uint64_t(1) << 32) * ((uint64_t(1) << sh) - uint64_t(ext))) / uint64_t(ext) + 1);
+    *shift = sh;
+}
+
+// Blocked form of a Wrap32Dev (natural tile order; tile strides from the extents).
+WrapTabDev make_wraptab(const Wrap32Dev& wd) {
+    WrapTabDev wt;
+    std::memset(&wt, 0, sizeof wt);
+    const int nd = wd.nd;
+    int64_t gst[2 * AOL_MAX_RANK];
+    int64_t g = 1;
+    for (int d = nd - 1; d >= 0; --d) {
+        gst[d] = g;
+        g *= wd.ext[d];
+    }
+    int k = nd - 1;
+    int64_t prod = 1;
+    while (k >= 0 && prod * wd.ext[k] <= kWTab) prod *= wd.ext[k--];
+    const int64_t c = k >= 0 ? std::max<int64_t>(1, kWTab / prod) : 1;
+    auto put_in = [&](int d, int64_t ext) {
+        wt.in_ext[wt.n_in] = int32_t(ext);
+        wt.in_lin[wt.n_in] = wd.lin[d];
+        wt.in_w0[wt.n_in] = wd.wc[0][d];
+        wt.in_w1[wt.n_in] = wd.wc[1][d];
+        magic32(ext, &wt.in_mul[wt.n_in], &wt.in_shift[wt.n_in]);
+        ++wt.n_in;
+    };
+    if (k >= 0) put_in(k, c);
+    for (int d = k + 1; d < nd; ++d) put_in(d, wd.ext[d]);
+    wt.inner = int32_t(prod * c);
+    wt.inner_tail = int32_t(prod);
+    wt.chunk_len = int32_t(c);
+    int64_t nblocks = 1;
+    auto put_out = [&](int64_t ext, int64_t lin, int64_t w0, int64_t w1, int64_t gs) {
+        wt.out_ext[wt.n_out] = int32_t(ext);
+        wt.out_lin[wt.n_out] = int32_t(lin);
+        wt.out_w0[wt.n_out] = int32_t(w0);
+        wt.out_w1[wt.n_out] = int32_t(w1);
+        wt.out_g[wt.n_out] = int32_t(gs);
+        magic32(ext, &wt.out_mul[wt.n_out], &wt.out_shift[wt.n_out]);
+        ++wt.n_out;
+        nblocks *= ext;
+    };
+    for (int d = 0; d < k; ++d) put_out(wd.ext[d], wd.lin[d], wd.wc[0][d], wd.wc[1][d], gst[d]);
+    const int64_t cext = k >= 0 ? wd.ext[k] : 1;
+    if (k >= 0)
+        put_out((cext + c - 1) / c, int64_t(wd.lin[k]) * c, int64_t(wd.wc[0][k]) * c, int64_t(wd.wc[1][k]) * c,
+                gst[k] * c);
+    else
+        put_out(1, 0, 0, 0, 0);
+    wt.chunk_ext = int32_t(cext);
+    wt.nblocks = int32_t(nblocks);
+    wt.base = wd.base;
+    wt.nw = wd.nw;
+    wt.worg0 = wd.worg[0];
+    wt.worg1 = wd.worg[1];
+    wt.wext0 = wd.wext[0];
+    wt.wext1 = wd.wext[1];
+    wt.wstep0 = wd.wstep[0];
+    wt.wstep1 = wd.wstep[1];
+    wt.wmul0 = wd.wmul[0];
+    wt.wshift0 = wd.wshift[0];
+    wt.wmul1 = wd.wmul[1];
+    wt.wshift1 = wd.wshift[1];
+    return wt;
+}
+
+// AOL_TILER_WRAPTAB=0 runs wrapping gathers / FAST scatters element by element (A/B measurements only).
+bool tiler_wraptab_enabled() {
+    static const bool v = [] {
+        const char* e = std::getenv("AOL_TILER_WRAPTAB");
+        return !(e && e[0] == '0');
+    }();
+    return v;
+}
+
 // AOL_TILER_WRAP32=0 keeps wrapping tilers on the 64-bit general kernel (A/B measurements only).
 bool tiler_wrap32_enabled() {
     static const bool v = [] {
@@ -412,6 +576,13 @@ aol_status_t launch_v(const TilerDev& td, const void* src, void* dst, unsigned l
             DeviceInfo dev;
             aol_status_t st = device_info(&dev);
             if (st != AOL_OK) return st;
+            if (MODE <= 1 && tiler_wraptab_enabled()) {
+                const WrapTabDev wt = make_wraptab(wd);
+                const int gt = int(std::max<int64_t>(1, std::min<int64_t>(wt.nblocks, int64_t(dev.num_sms) * 8)));
+                tiler_wraptab_kernel<ES, MODE><<<gt, 256, 0, s>>>(wt, src, dst);
+                AOL_LAUNCH_CHECK("tiler_wraptab_kernel");
+                return AOL_OK;
+            }
             const int gw = int(std::max<int64_t>(1, std::min<int64_t>((td.total + 255) / 256, int64_t(dev.num_sms) * 128)));
             tiler_wrap32_kernel<ES, MODE><<<gw, 256, 0, s>>>(wd, src, dst, ws);
             AOL_LAUNCH_CHECK("tiler_wrap32_kernel");

@@ -42,7 +42,7 @@ cases = {
     "d3 8x8 blocks wrapping": ([64, 1024, 1024], [64, 128, 128], [8, 8], [0, -3, 5], [[1, 0, 0], [0, 8, 0], [0, 0, 8]],
                                [[0, 0], [1, 0], [0, 1]], (64, 128, 128, 8, 8)),
 }
-tag = {"wrap32": os.environ.get("AOL_TILER_WRAP32", "1")}
+tag = {"wrap32": os.environ.get("AOL_TILER_WRAP32", "1"), "wraptab": os.environ.get("AOL_TILER_WRAPTAB", "1")}
 for name, (arr, rep, pat, o, P, F, gshape) in cases.items():
     t = aol.make_tiler(arr, rep, pat, o, P, F)
     G = torch.empty(gshape, dtype=torch.int32, device="cuda")
