@@ -17,6 +17,7 @@ from typing import Optional, Sequence
 import torch
 
 from . import _lib
+from ._lib import FLAGS  # noqa: F401  (launch-option flag bits, include/aol.h AOL_FLAG_*)
 from ._lib import (FILTER_H, FILTER_V, AolError, I16, I32, I64, PRESET_H_IN, PRESET_H_OUT, PRESET_V_IN,
                    PRESET_V_OUT, RAW8, RAW16, RAW32, RAW64, SCATTER_FAST, SCATTER_SEQUENTIAL, U8, aol_filter_t,
                    aol_launch_opts_t, aol_plan_t, aol_tiler_t, check, lib)
@@ -26,7 +27,7 @@ __all__ = [
     "tiler_gather", "tiler_scatter", "downscale_h", "downscale_v", "downscale_frame", "downscale_frame_plan",
     "frame_checksum", "downscale_frame_host", "synth_frames", "library_path",
     "PRESET_H_IN", "PRESET_H_OUT", "PRESET_V_IN", "PRESET_V_OUT", "SYNTH_KINDS",
-    "make_filter", "filter_preset", "filter_validate", "filter_apply", "FILTER_H", "FILTER_V",
+    "make_filter", "filter_preset", "filter_validate", "filter_apply", "FILTER_H", "FILTER_V", "FLAGS",
 ]
 
 SYNTH_KINDS = {"uniform": 0, "dark": 1, "signed": 2, "ramp": 3, "constant": 4}

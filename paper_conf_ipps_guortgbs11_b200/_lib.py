@@ -57,6 +57,16 @@ class aol_filter_t(ctypes.Structure):
                 ("window_start", ctypes.c_int32 * MAX_WINDOWS)]
 
 
+# aol_launch_opts_t.flags bits (include/aol.h AOL_FLAG_*; tuning experiments, results are identical)
+FLAG_EVICT_FIRST_LOADS, FLAG_EVICT_FIRST_STORES, FLAG_BLOCKED_UNITS, FLAG_U8_BULK = 2, 4, 8, 16
+FLAG_U8_ONE_REP, FLAG_NO_PDL, FLAG_I32_LINEAR, FLAG_I32_SWZ32 = 32, 64, 128, 256
+FLAG_ROW_STAGES, FLAG_TRIPLE_STAGES = 512, 1024
+FLAGS = {"EVICT_FIRST_LOADS": FLAG_EVICT_FIRST_LOADS, "EVICT_FIRST_STORES": FLAG_EVICT_FIRST_STORES,
+         "BLOCKED_UNITS": FLAG_BLOCKED_UNITS, "U8_BULK": FLAG_U8_BULK, "U8_ONE_REP": FLAG_U8_ONE_REP,
+         "NO_PDL": FLAG_NO_PDL, "I32_LINEAR": FLAG_I32_LINEAR, "I32_SWZ32": FLAG_I32_SWZ32,
+         "ROW_STAGES": FLAG_ROW_STAGES, "TRIPLE_STAGES": FLAG_TRIPLE_STAGES}
+
+
 class aol_launch_opts_t(ctypes.Structure):
     _fields_ = [("ctas_per_sm", ctypes.c_int32), ("stages", ctypes.c_int32),
                 ("bands_per_unit", ctypes.c_int32), ("kernel", ctypes.c_int32),

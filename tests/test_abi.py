@@ -244,3 +244,19 @@ def test_c_example_builds_against_header():
                            "-L", os.path.dirname(_lib.LIB_PATH), "-laol", "-L", "/usr/local/cuda/lib64", "-lcudart",
                            "-o", out])
     assert os.path.exists(out)
+
+
+def test_binding_constants_match_header():
+    """The Python binding's enum and flag values are the ones include/aol.h declares (marshalling only:
+    a drifted constant would silently select another dtype, preset or launch option)."""
+    import re
+
+    hdr = open(os.path.join(ROOT, "include", "aol.h")).read()
+    flags = {m.group(1): int(m.group(2)) for m in re.finditer(r"#define AOL_FLAG_(\w+)\s+(\d+)", hdr)}
+    assert flags == aol.FLAGS
+    for name, val in (("AOL_U8", _lib.U8), ("AOL_I16", _lib.I16), ("AOL_I32", _lib.I32), ("AOL_I64", _lib.I64),
+                      ("AOL_RAW8", _lib.RAW8), ("AOL_RAW64", _lib.RAW64), ("AOL_PRESET_V_OUT", _lib.PRESET_V_OUT),
+                      ("AOL_SCATTER_SEQUENTIAL", _lib.SCATTER_SEQUENTIAL), ("AOL_FILTER_V", _lib.FILTER_V),
+                      ("AOL_E_CUDA", -7)):
+        m = re.search(name + r"\s*=\s*(-?\d+)", hdr)
+        assert m and int(m.group(1)) == val, name
