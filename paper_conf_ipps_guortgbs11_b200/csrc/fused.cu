@@ -17,10 +17,15 @@ using namespace fused;
 
 namespace {
 
-// Zeroes the per-frame checksums ahead of a fused launch.  It lets that launch start at once
+// Zeroes the per-frame checksums ahead of a fused launch.  It is itself launched as a programmatic dependent
+// of whatever precedes it in the stream (the previous fused kernel triggers its dependents at its start), so
+// its one CTA is already resident when that kernel drains; griddepcontrol.wait then holds it until the
+// preceding grid has completed and its writes are visible (the previous call may still be adding into the
+// same checksums, or producing X).  Only after that wait does it let the fused launch start
 // (griddepcontrol.launch_dependents): the fused kernel's prologue, TMA ring fill and whole first work unit
-// overlap this kernel, and only its first checksum atomic waits for it (ptx::griddep_wait).
+// overlap the zeroing, and only its first checksum atomic waits for it (ptx::griddep_wait).
 __global__ void __launch_bounds__(256) zero_checksums_kernel(uint64_t* __restrict__ cs, int64_t n) {
+    ptx::griddep_wait();
     ptx::griddep_launch_dependents();
     for (int64_t i = threadIdx.x; i < n; i += blockDim.x) cs[i] = 0;
 }
@@ -336,8 +341,23 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
     // dependent, so the zeroing (and the launch gap after it) overlaps the fused kernel's start instead of
     // preceding it (single-frame latency).  Only the zero kernel can be the primary: it
     // is an ordinary launch, so everything earlier in the stream (e.g. the producer of X) has completed.
+    const bool pdl = d_cs && !(plan.flags & AOL_FLAG_NO_PDL);
     if (d_cs) {
-        zero_checksums_kernel<<<1, 256, 0, s>>>(d_cs, frames);
+        cudaLaunchConfig_t zc;
+        std::memset(&zc, 0, sizeof zc);
+        zc.gridDim = dim3(1);
+        zc.blockDim = dim3(256);
+        zc.stream = s;
+        cudaLaunchAttribute za[1];
+        za[0].id = cudaLaunchAttributeProgrammaticStreamSerialization;
+        za[0].val.programmaticStreamSerializationAllowed = 1;
+        zc.attrs = za;
+        zc.numAttrs = pdl ? 1 : 0;
+        cudaError_t ze = cudaLaunchKernelEx(&zc, zero_checksums_kernel, d_cs, int64_t(frames));
+        if (ze != cudaSuccess) {
+            set_error("launch of zero_checksums_kernel failed: %s", cudaGetErrorString(ze));
+            return AOL_E_CUDA;
+        }
         AOL_LAUNCH_CHECK("zero_checksums_kernel");
     }
     cudaLaunchConfig_t cfg;
@@ -350,7 +370,7 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
     attr[0].id = cudaLaunchAttributeProgrammaticStreamSerialization;
     attr[0].val.programmaticStreamSerializationAllowed = 1;
     cfg.attrs = attr;
-    cfg.numAttrs = (d_cs && !(plan.flags & AOL_FLAG_NO_PDL)) ? 1 : 0;
+    cfg.numAttrs = pdl ? 1 : 0;
     cudaError_t le = cudaLaunchKernelEx(&cfg, k, map, a);
     if (le != cudaSuccess) {
         set_error("launch of fused_tma_kernel failed: %s", cudaGetErrorString(le));

@@ -234,6 +234,9 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
     uint64_t* empty = full + a.stages;
     unsigned long long* red = reinterpret_cast<unsigned long long*>(empty + a.stages);   // [32] checksum partials
 
+    // Let a programmatic dependent of this launch (the next call's checksum-zeroing kernel, which waits for
+    // this grid's completion before touching anything) become resident now instead of after the drain.
+    ptx::griddep_launch_dependents();
     const int tid = threadIdx.x;
     const int NC = a.n_consumer;
     if (tid == 0) {

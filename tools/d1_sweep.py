@@ -36,8 +36,11 @@ def graph_us(x, z, cs, opts, fn=None):
 x = aol.synth_frames(0, 0, 1, 3, 1080, 1920)
 z = torch.empty((1, 3, 480, 720), dtype=torch.int32, device="cuda")
 cs = torch.empty(1, dtype=torch.uint64, device="cuda")
-for opts in [None, {"flags": 64}, {"ctas_per_sm": 2, "bands_per_unit": 1, "flags": 64}, {"ctas_per_sm": 2}, {"ctas_per_sm": 2, "bands_per_unit": 1}, {"ctas_per_sm": 2, "bands_per_unit": 2},
-             {"ctas_per_sm": 3, "bands_per_unit": 1}, {"bands_per_unit": 1}, {"bands_per_unit": 2}, {"stages": 3}]:
+for opts in [None, {"flags": 64}, {"ctas_per_sm": 2}, {"ctas_per_sm": 2, "bands_per_unit": 1}, {"ctas_per_sm": 2, "bands_per_unit": 2},
+             {"ctas_per_sm": 3, "bands_per_unit": 1}, {"bands_per_unit": 1}, {"bands_per_unit": 2}, {"stages": 3},
+             {"flags": 512}, {"flags": 512, "stages": 8}, {"flags": 512, "ctas_per_sm": 2, "bands_per_unit": 1},
+             {"flags": 512, "ctas_per_sm": 2, "bands_per_unit": 2}, {"flags": 512, "ctas_per_sm": 3, "bands_per_unit": 1},
+             {"flags": 128}, {"flags": 128 | 512, "ctas_per_sm": 2, "bands_per_unit": 1}]:
     us = graph_us(x, z, cs, opts)
     print(json.dumps({"opts": opts, "us_per_call": us, "plan": aol.downscale_frame_plan(1, 3, 1080, 1920, opts=opts)}))
 
