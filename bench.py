@@ -105,6 +105,23 @@ def ncu_traffic(a):
         return None, None, None
 
 
+def mix_ceiling(a):
+    """Best rate the committed HBM probe (tools/hbm_probe.cu: an idealised TMA streamer, no compute) reached
+    for this path's read:write byte mix -- what this GPU's HBM delivers for that mix, as opposed to the copy
+    peak (half writes).  (GB/s, source) or (None, None)."""
+    if a.dtype == "i32":
+        f, wpm = "r01_hbm_probe_inter.jsonl", 166
+    else:
+        f, wpm = "r01_hbm_probe_u8.jsonl", 333 if a.out_dtype == "i16" else 666
+    try:
+        with open(os.path.join(ROOT, "profiles", f)) as fh:
+            rows = [json.loads(line) for line in fh if line.strip()]
+        best = max(r["GBps"] for r in rows if r.get("write_permille") == wpm)
+        return best, f"profiles/{f} (best over chunk size x ring depth x CTAs/SM, write/read = {wpm}/1000)"
+    except Exception:
+        return None, None
+
+
 class ClockSampler:
     """Samples SM clocks and throttle reasons with NVML during the timed region."""
 
@@ -365,6 +382,8 @@ def main():
     achieved = bpf * sum(launch_frames) / (sum(launch_ms) / 1000.0) / 1e9
     peak, peak_src = measured_peak()
     traffic, dram_pct, ncu_tag = ncu_traffic(a)
+    mix_gbs, mix_src = mix_ceiling(a)
+    mix = ({"GBps": mix_gbs, "frac": achieved / mix_gbs, "source": mix_src} if mix_gbs else None)
     line = {
         "metric": METRIC, "value": value, "unit": "frames/s", "n_gpus": world, "steps": a.steps,
         "warmup": a.warmup, "ms_per_step": max_ms / a.steps, "higher_is_better": True,
@@ -381,6 +400,7 @@ def main():
                      # the copy peak is half writes while this path is ~86 % reads, so frac can exceed 1; ncu's
                      # DRAM utilisation of the same launch (committed capture) is the direct measure
                      "ncu_dram_pct_of_peak": dram_pct, "ncu_capture": ncu_tag,
+                     "mix_ceiling": mix,
                      "algorithmic_bytes_per_launch": bpf * calls[0],
                      "avg_launch_ms": avg_launch_s * 1000.0, "min_launch_ms": min(launch_ms)},
         # per call: zero_checksums_kernel + the fused kernel (its programmatic dependent)
