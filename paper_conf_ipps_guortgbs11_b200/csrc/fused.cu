@@ -6,7 +6,6 @@
 #include <algorithm>
 #include <cstdint>
 #include <cstring>
-#include <vector>
 
 #include "common.h"
 #include "fused_kernel.cuh"
@@ -205,8 +204,8 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void*
     }
     if (o.kernel == 1 && !tma_ok) {
         set_error("TMA fused kernel requested but unsupported for this shape/dtype/alignment "
-                  "(W <= 7936 and a 2-stage ring within shared memory; int32 with W %% 32 == 0: W <= 7680; "
-                  "uint8: W %% 16 == 0; 16-byte aligned buffers)");
+                  "(W <= 7936 and a 2-stage ring within shared memory; uint8: W %% 16 == 0; 16-byte aligned "
+                  "buffers)");
         return AOL_E_SHAPE;
     }
     if (o.kernel == 2) tma_ok = false;
@@ -225,19 +224,20 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void*
             // at 8; profiles/r01_nb_sweep.jsonl).
             // (int16 outputs run 3 CTAs/SM: the epilogue weighs ~1.5x more; HD 0.421 ms at 20 vs 0.425 at 15)
             const double ovh = in_dtype == AOL_U8 ? (out_es == 2 ? 5760.0 : 3840.0) / double(W) : 0.0;
-            const int max_nb = std::min(nbands, 120);
-            std::vector<double> cost(size_t(max_nb) + 1, 0.0);
+            constexpr int kMaxNb = 120;
+            const int max_nb = std::min(nbands, kMaxNb);
+            double cost[kMaxNb + 1] = {};
             double best = 1e300;
             for (int cand = 1; cand <= max_nb; ++cand) {
                 const int64_t units = planes * ((nbands + cand - 1) / cand);
                 const int64_t waves = (units + max_ctas - 1) / max_ctas;
-                cost[size_t(cand)] = double(waves) * (3.0 * cand + 1.0 + ovh);
-                best = std::min(best, cost[size_t(cand)]);
+                cost[cand] = double(waves) * (3.0 * cand + 1.0 + ovh);
+                best = std::min(best, cost[cand]);
             }
             for (int cand = 1; cand <= max_nb; ++cand) {
                 if (in_dtype == AOL_U8) {
-                    if (cost[size_t(cand)] <= best) nb = cand;   // largest of the cheapest
-                } else if (cost[size_t(cand)] <= 1.02 * best) {
+                    if (cost[cand] <= best) nb = cand;   // largest of the cheapest
+                } else if (cost[cand] <= 1.02 * best) {
                     nb = cand;                                   // smallest within 2 %
                     break;
                 }
