@@ -271,7 +271,10 @@ def main():
     torch.cuda.set_device(gpu)
     dev = torch.device("cuda", gpu)
     backend = os.environ.get("AOL_DIST_BACKEND", "nccl")
-    if world > 1:
+    # AOL_FORCE_DIST=1: join a process group even as a single rank (exercises the NCCL barrier / max-reduce /
+    # checksum all-gather code on a one-GPU box; the GPU tests use it)
+    use_dist = world > 1 or os.environ.get("AOL_FORCE_DIST") == "1"
+    if use_dist:
         if backend == "nccl":
             dist.init_process_group("nccl", device_id=dev)
         else:
@@ -315,7 +318,7 @@ def main():
     ends = [[torch.cuda.Event(enable_timing=True) for _ in calls] for _ in range(a.steps)]
     t_begin = torch.cuda.Event(enable_timing=True)
     t_end = torch.cuda.Event(enable_timing=True)
-    if world > 1:
+    if use_dist:
         dist.barrier()
     torch.cuda.synchronize(dev)
     with ClockSampler(gpu) as clk:
@@ -324,7 +327,7 @@ def main():
             step((starts[i], ends[i]))
         t_end.record(stream)
         torch.cuda.synchronize(dev)
-    if world > 1:
+    if use_dist:
         dist.barrier()
     elapsed_ms = t_begin.elapsed_time(t_end)
     launch_ms = [s.elapsed_time(e) for ss, es in zip(starts, ends) for s, e in zip(ss, es)]
@@ -334,7 +337,7 @@ def main():
     counts = ([max(1, min(a.pool, shard.strong_range(r, world, a.stream_frames)[1])) for r in range(world)]
               if a.stream_frames else None)
     max_ms, cs_all_t = shard.gather_results(cs if backend == "nccl" else cs.cpu(), elapsed_ms, counts=counts)
-    cs_all = cs_all_t.cpu().numpy().view(np.uint64) if world > 1 else None
+    cs_all = cs_all_t.cpu().numpy().view(np.uint64) if use_dist else None
     if a.dump_checksums and rank == 0:
         np.save(a.dump_checksums, cs_all if cs_all is not None else cs.cpu().view(torch.int64).numpy().view(np.uint64))
 
@@ -351,7 +354,7 @@ def main():
         ws = torch.empty(aol.host_workspace_bytes(chunk, C, H, W, tdtype), dtype=torch.uint8, device=dev)
         streams = [torch.cuda.Stream(device=dev) for _ in range(3)]
         aol.downscale_frame_host(x_host, out=z_host, chunk_frames=chunk, workspace=ws, streams=streams, device=dev)
-        if world > 1:
+        if use_dist:
             dist.barrier()
         t0 = time.perf_counter()
         for _ in range(a.e2e_steps):
@@ -359,7 +362,7 @@ def main():
                                                streams=streams, device=dev)
         e2e_s = time.perf_counter() - t0
         te = torch.tensor([e2e_s], dtype=torch.float64, device=dev if backend == "nccl" else "cpu")
-        if world > 1:
+        if use_dist:
             dist.all_reduce(te, op=dist.ReduceOp.MAX)
         e2e_s = float(te.item())
         same = bool(torch.equal(cs_h.view(torch.int64), cs[:Fe].cpu().view(torch.int64)))
@@ -370,7 +373,7 @@ def main():
                "timing": "host wall clock around the blocking call, max over ranks"}
 
     if rank != 0:
-        if world > 1:
+        if use_dist:
             dist.destroy_process_group()
         return
 
@@ -409,7 +412,7 @@ def main():
     }
     if e2e is not None:
         line["e2e"] = e2e
-    if world > 1 and cs_all is not None:
+    if use_dist and cs_all is not None:
         line["gathered_checksums"] = int(cs_all.size)
     if world == 1 and not a.no_cpu_baseline:
         fps, info = cpu_baseline(a, gpu_cs=cs.cpu().view(torch.int64).numpy().view(np.uint64), frame0=frame0,
@@ -417,7 +420,7 @@ def main():
         line["cpu_baseline"] = {"value": fps, "unit": "frames/s", "cores": info["cores"], "kind": "oracle",
                                 "sample": info["sample"], "parity_sample_ok": info.get("parity_sample_ok")}
     print(json.dumps(line), flush=True)
-    if world > 1:
+    if use_dist:
         dist.destroy_process_group()
 
 

@@ -39,11 +39,11 @@ def gather_results(checksums: torch.Tensor, elapsed_ms: float, group: Optional[d
     backend's device).  counts: per-rank frame counts when ranks hold different
     numbers of frames (strong scaling); default = equal counts.
     Returns (max_elapsed_ms, int64 tensor of all checksums on the same device)."""
-    world = dist.get_world_size(group) if dist.is_initialized() else 1
     cs = checksums.view(torch.int64) if checksums.dtype == torch.uint64 else checksums.to(torch.int64)
     t = torch.tensor([float(elapsed_ms)], dtype=torch.float64, device=cs.device)
-    if world == 1:
+    if not dist.is_initialized():   # single process: nothing to exchange
         return float(t.item()), cs.clone()
+    world = dist.get_world_size(group)
     dist.all_reduce(t, op=dist.ReduceOp.MAX, group=group)
     if counts is None:
         out = torch.empty(world * cs.numel(), dtype=torch.int64, device=cs.device)

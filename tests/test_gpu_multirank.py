@@ -57,3 +57,25 @@ def test_strong_stream_two_ranks(orc, tmp_path):
     _, ref0 = orc.downscale_frame(synth.frames(0, 0, 4, C, H, W), nthreads=8)
     _, ref1 = orc.downscale_frame(synth.frames(0, 12, 4, C, H, W), nthreads=8)
     assert np.array_equal(cs, np.concatenate([ref0, ref1]))
+
+
+@pytest.mark.parametrize("mode", ["weak", "strong"])
+def test_nccl_collectives_single_rank(orc, tmp_path, mode):
+    """The NCCL code path of the multi-GPU bench (process group on the GPU, barrier, float64 MAX all-reduce,
+    int64 checksum all-gather incl. the ragged strong-scaling gather) as a single rank on this one-GPU box
+    (AOL_FORCE_DIST=1; NCCL cannot put two ranks on one GPU), checksums against the oracle."""
+    dump = str(tmp_path / "cs.npy")
+    env = dict(os.environ, AOL_FORCE_DIST="1")
+    env.pop("AOL_DIST_BACKEND", None)
+    extra = ["--frames", "4"] if mode == "weak" else ["--stream-frames", "7", "--pool", "3"]
+    cmd = [sys.executable, "-m", "torch.distributed.run", "--nnodes=1", "--nproc-per-node", "1",
+           "--master-addr", "127.0.0.1", "--master-port", str(_port()), os.path.join(ROOT, "bench.py"),
+           "--H", str(H), "--W", str(W), "--steps", "3", "--warmup", "3", "--no-cpu-baseline",
+           "--dump-checksums", dump, *extra]
+    r = subprocess.run(cmd, capture_output=True, text=True, timeout=600, cwd=ROOT, env=env)
+    assert r.returncode == 0, r.stderr[-3000:]
+    d = json.loads([l for l in r.stdout.strip().splitlines() if l.startswith("{")][-1])
+    n = 4 if mode == "weak" else 3
+    assert d["gathered_checksums"] == n and d["value"] > 0
+    _, ref = orc.downscale_frame(synth.frames(0, 0, n, C, H, W), nthreads=8)
+    assert np.array_equal(np.load(dump), ref)
