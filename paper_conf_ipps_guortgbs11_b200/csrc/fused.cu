@@ -5,6 +5,7 @@
 
 #include <algorithm>
 #include <cstdint>
+#include <cstdlib>
 #include <cstring>
 
 #include "common.h"
@@ -115,6 +116,20 @@ int smem_bytes(const RingGeom& g, int stages) {
     return stages * int(g.stage_stride) + kOutBufs * int(g.out_bytes) + 2 * stages * 8 + 256 + 1024;
 }
 
+// L2 sector promotion of the TMA loads: none (the rows are streamed once; 256-byte promotion measured 0.2-0.4 %
+// slower on HD / 4K int32 and HD uint8, profiles/r01_l2promo_ab.jsonl).  AOL_TMA_L2_PROMO=1/2/3 selects
+// 64 / 128 / 256 B (A/B measurements only).
+CUtensorMapL2promotion l2_promotion() {
+    static const CUtensorMapL2promotion v = [] {
+        const char* e = std::getenv("AOL_TMA_L2_PROMO");
+        if (e && e[0] == '1') return CU_TENSOR_MAP_L2_PROMOTION_L2_64B;
+        if (e && e[0] == '2') return CU_TENSOR_MAP_L2_PROMOTION_L2_128B;
+        if (e && e[0] == '3') return CU_TENSOR_MAP_L2_PROMOTION_L2_256B;
+        return CU_TENSOR_MAP_L2_PROMOTION_NONE;
+    }();
+    return v;
+}
+
 // TMA descriptor for row triples of a [rows][W] array viewed as {inner, W/inner, rows}: int32 with a
 // 128 B swizzle (inner = 32 elements), uint8 unswizzled (inner = 128 elements).
 aol_status_t encode_row_map(CUtensorMap* map, aol_dtype_t dt, const void* base, int64_t rows, int64_t W, int flags) {
@@ -131,7 +146,7 @@ aol_status_t encode_row_map(CUtensorMap* map, aol_dtype_t dt, const void* base, 
     CUresult cr = encode(map, i32 ? CU_TENSOR_MAP_DATA_TYPE_INT32 : CU_TENSOR_MAP_DATA_TYPE_UINT8, 3,
                          const_cast<void*>(base), gdim, gstride, box, estr, CU_TENSOR_MAP_INTERLEAVE_NONE,
                          i32 ? (s32 ? CU_TENSOR_MAP_SWIZZLE_32B : CU_TENSOR_MAP_SWIZZLE_128B) : CU_TENSOR_MAP_SWIZZLE_NONE,
-                         CU_TENSOR_MAP_L2_PROMOTION_L2_256B, CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+                         l2_promotion(), CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
     if (cr != CUDA_SUCCESS) {
         set_error("cuTensorMapEncodeTiled failed (CUresult %d)", int(cr));
         return AOL_E_CUDA;
