@@ -1,0 +1,637 @@
+// tiler_kernels.cuh -- the generic tiler kernels and their per-element-size launchers, compiled once per
+// element size (tiler_es{1,2,4,8}.cu, in parallel); tiler.cu holds the host entry points.
+// K-1 generic ArrayOL tiler gather and K-2 scatter (any rank <= 8,
+// element size 1/2/4/8 bytes, Euclidean modulo).
+//
+//   gather : tiles[r][i]  = array[(o + P.r + F.i) mod s]     (Section IV, Fig. 4)
+//   scatter: array[(o + P.r + F.i) mod s] = tiles[r][i]      (Fig. 6, modarray P:L479)
+//
+// The host reduces o, P and F modulo the array extents (every partial sum is
+// then non-negative) and classifies each array dimension: if no (r, i) can
+// push its coordinate past the extent, the `mod` is the identity there.  When
+// that holds for every dimension the tiler is an affine map of the flat tile
+// index -- offset = base + sum_d lin[d] * idx[d] -- and the LINEAR kernels
+// apply: one fast 32-bit division chain per thread and, when the innermost
+// pattern dimension walks contiguous memory, 16-byte vector accesses on both
+// sides.  Linear tilers are walked in array-stride order (the host sorts the
+// combined dims so consecutive threads touch consecutive ARRAY addresses, the
+// side whose locality is not guaranteed); the tile side is then written in
+// contiguous runs of the innermost dim.  Otherwise the GENERAL kernels walk the
+// natural tile order (tile accesses coalesced) and evaluate the modulo per
+// wrapping dimension.
+#pragma once
+#include <cuda_runtime.h>
+
+#include <algorithm>
+#include <cstdint>
+#include <cstdlib>
+#include <cstring>
+
+#include "common.h"
+
+namespace aol {
+
+namespace {
+
+template <int ES>
+struct Elem;
+template <>
+struct Elem<1> {
+    using T = uint8_t;
+};
+template <>
+struct Elem<2> {
+    using T = uint16_t;
+};
+template <>
+struct Elem<4> {
+    using T = uint32_t;
+};
+template <>
+struct Elem<8> {
+    using T = unsigned long long;
+};
+
+template <int BYTES>
+struct Vec;
+template <>
+struct Vec<1> {
+    using T = uint8_t;
+};
+template <>
+struct Vec<2> {
+    using T = uint16_t;
+};
+template <>
+struct Vec<4> {
+    using T = uint32_t;
+};
+template <>
+struct Vec<8> {
+    using T = uint2;
+};
+template <>
+struct Vec<16> {
+    using T = uint4;
+};
+
+constexpr int kND = 2 * AOL_MAX_RANK;
+
+// Decompose flat index g over extents ext (last dim fastest).
+template <bool kFast32>
+__device__ __forceinline__ void decompose(int nd, const int64_t* ext, const uint32_t* fmul, const uint32_t* fshift,
+                                          int64_t g, int64_t (&idx)[kND]) {
+#pragma unroll
+    for (int d = kND - 1; d >= 0; --d) {
+        if (d < nd) {
+            if (kFast32) {
+                const uint32_t n = uint32_t(g);
+                const uint32_t q = (__umulhi(n, fmul[d]) + n) >> fshift[d];
+                idx[d] = int64_t(n - q * uint32_t(ext[d]));
+                g = q;
+            } else {
+                const int64_t q = g / ext[d];
+                idx[d] = g - q * ext[d];
+                g = q;
+            }
+        } else {
+            idx[d] = 0;
+        }
+    }
+}
+
+__device__ __forceinline__ int64_t general_offset(const TilerDev& td, const int64_t (&idx)[kND]) {
+    int64_t off = 0;
+#pragma unroll
+    for (int a = 0; a < AOL_MAX_RANK; ++a) {
+        if (a < td.ra) {
+            int64_t v = td.org[a];
+#pragma unroll
+            for (int d = 0; d < kND; ++d)
+                if (d < td.nd) v += td.coef[a][d] * idx[d];
+            if (!((td.nowrap_mask >> a) & 1)) v %= td.ashape[a];   // all terms >= 0: % == Euclidean mod
+            off += v * td.astride[a];
+        }
+    }
+    return off;
+}
+
+// mode 0: gather; 1: FAST scatter; 2: SEQUENTIAL claim (max flat index + 1 per target);
+// 3: SEQUENTIAL write (store iff this element holds the claim).
+template <int ES, int V, bool kFast32, bool kLinear, int MODE>
+__global__ void __launch_bounds__(256) tiler_kernel(const TilerDev td, const void* __restrict__ src,
+                                                    void* __restrict__ dst, unsigned long long* __restrict__ ws) {
+    using T = typename Elem<ES>::T;
+    using VT = typename Vec<ES * V>::T;
+    const int64_t nvec = td.total / V;
+    const int64_t stride = int64_t(gridDim.x) * blockDim.x;
+    // kU independent elements per thread per iteration: all loads issued before the stores, so each
+    // thread keeps kU requests in flight (Little's law at ~43 GB/s per SM needs tens of KB per SM).
+    constexpr int kU = (MODE <= 1) ? 4 : 1;
+    // a warp owns kU*32 consecutive vectors per iteration (lane + 32u): locality is kept on both sides
+    const int64_t warp_first = (int64_t(blockIdx.x) * blockDim.x + (threadIdx.x & ~31u)) * kU + (threadIdx.x & 31u);
+    for (int64_t v0 = warp_first; v0 < nvec; v0 += kU * stride) {
+        int64_t off[kU], g[kU];   // array-side and tile-side element offsets
+#pragma unroll
+        for (int u = 0; u < kU; ++u) {
+            const int64_t v = v0 + 32 * u;
+            if (kLinear) {
+                // permuted walk (array side contiguous): both offsets are affine in the permuted index;
+                // a runtime-rank loop that folds each digit straight into the two offsets (no index array)
+                int64_t o = td.base, gg = 0;
+                if (kFast32) {
+                    uint32_t n = v < nvec ? uint32_t(v * V) : 0u;
+#pragma unroll 1
+                    for (int d = td.nd - 1; d >= 0; --d) {
+                        const uint32_t q = (__umulhi(n, td.p_fd_mul[d]) + n) >> td.p_fd_shift[d];
+                        const uint32_t i = n - q * uint32_t(td.p_ext[d]);
+                        n = q;
+                        o += td.p_lin[d] * int64_t(i);
+                        gg += td.p_gst[d] * int64_t(i);
+                    }
+                } else {
+                    int64_t n = v < nvec ? v * V : 0;
+#pragma unroll 1
+                    for (int d = td.nd - 1; d >= 0; --d) {
+                        const int64_t q = n / td.p_ext[d];
+                        const int64_t i = n - q * td.p_ext[d];
+                        n = q;
+                        o += td.p_lin[d] * i;
+                        gg += td.p_gst[d] * i;
+                    }
+                }
+                off[u] = o;
+                g[u] = gg;
+            } else {
+                int64_t idx[kND];
+                g[u] = v < nvec ? v * V : 0;
+                decompose<kFast32>(td.nd, td.ext, td.fd_mul, td.fd_shift, g[u], idx);
+                off[u] = general_offset(td, idx);
+            }
+        }
+        if (MODE == 0) {
+            // tiles[g .. g+V) = array[off .. off+V)   (V > 1 only when contiguous and aligned)
+            VT val[kU];
+#pragma unroll
+            for (int u = 0; u < kU; ++u)
+                if (v0 + 32 * u < nvec) val[u] = reinterpret_cast<const VT*>(static_cast<const T*>(src) + off[u])[0];
+#pragma unroll
+            for (int u = 0; u < kU; ++u)
+                if (v0 + 32 * u < nvec) reinterpret_cast<VT*>(static_cast<T*>(dst) + g[u])[0] = val[u];
+        } else if (MODE == 1) {
+            VT val[kU];
+#pragma unroll
+            for (int u = 0; u < kU; ++u)
+                if (v0 + 32 * u < nvec) val[u] = reinterpret_cast<const VT*>(static_cast<const T*>(src) + g[u])[0];
+#pragma unroll
+            for (int u = 0; u < kU; ++u)
+                if (v0 + 32 * u < nvec) reinterpret_cast<VT*>(static_cast<T*>(dst) + off[u])[0] = val[u];
+        } else if (MODE == 2) {
+            atomicMax(ws + off[0], (unsigned long long)g[0] + 1ull);
+        } else {
+            if (ws[off[0]] == (unsigned long long)g[0] + 1ull)
+                static_cast<T*>(dst)[off[0]] = static_cast<const T*>(src)[g[0]];
+        }
+    }
+}
+
+// Linear tilers whose array and tile offsets fit in 31 bits (the common case): the permuted walk with
+// all-32-bit digit arithmetic and the per-dimension constants staged once per CTA in shared memory
+// (one LDS.128 + one LDS per digit instead of five dynamically indexed constant-bank loads).
+template <int ES, int V, int MODE>
+__global__ void __launch_bounds__(256) tiler_linear32_kernel(const TilerDev td, const void* __restrict__ src,
+                                                             void* __restrict__ dst) {
+    using T = typename Elem<ES>::T;
+    using VT = typename Vec<ES * V>::T;
+    __shared__ int4 pk[kND];      // {extent, magic multiplier, shift, array stride}
+    __shared__ int32_t pg[kND];   // tile stride
+    if (threadIdx.x < td.nd) {
+        const int d = threadIdx.x;
+        pk[d] = make_int4(int32_t(td.p_ext[d]), int32_t(td.p_fd_mul[d]), int32_t(td.p_fd_shift[d]),
+                          int32_t(td.p_lin[d]));
+        pg[d] = int32_t(td.p_gst[d]);
+    }
+    __syncthreads();
+    const int32_t nvec = int32_t(td.total / V);
+    const int32_t stride = int32_t(gridDim.x * blockDim.x);
+    // 2 vectors per thread per iteration with a 4x larger grid than the general kernels (tools/tiler_probe2.py,
+    // profiles/r01_tiler_variants.jsonl: d3 gather 5.01 -> 5.22 TB/s; kU = 1, 4, 8 and grids x8..x512 are slower)
+    constexpr int kU = 2;
+    const int32_t warp_first = int32_t((blockIdx.x * blockDim.x + (threadIdx.x & ~31u)) * kU + (threadIdx.x & 31u));
+    for (int32_t v0 = warp_first; v0 < nvec; v0 += kU * stride) {
+        int32_t off[kU], g[kU];
+#pragma unroll
+        for (int u = 0; u < kU; ++u) {
+            const int32_t v = v0 + 32 * u;
+            uint32_t n = v < nvec ? uint32_t(v) * V : 0u;
+            int32_t o = int32_t(td.base), gg = 0;
+#pragma unroll 1
+            for (int d = td.nd - 1; d >= 0; --d) {
+                const int4 p = pk[d];
+                const uint32_t q = (__umulhi(n, uint32_t(p.y)) + n) >> p.z;
+                const int32_t i = int32_t(n - q * uint32_t(p.x));
+                n = q;
+                o += p.w * i;
+                gg += pg[d] * i;
+            }
+            off[u] = o;
+            g[u] = gg;
+        }
+        VT val[kU];
+        if (MODE == 0) {
+#pragma unroll
+            for (int u = 0; u < kU; ++u)
+                if (v0 + 32 * u < nvec) val[u] = reinterpret_cast<const VT*>(static_cast<const T*>(src) + off[u])[0];
+#pragma unroll
+            for (int u = 0; u < kU; ++u)
+                if (v0 + 32 * u < nvec) reinterpret_cast<VT*>(static_cast<T*>(dst) + g[u])[0] = val[u];
+        } else {
+#pragma unroll
+            for (int u = 0; u < kU; ++u)
+                if (v0 + 32 * u < nvec) val[u] = reinterpret_cast<const VT*>(static_cast<const T*>(src) + g[u])[0];
+#pragma unroll
+            for (int u = 0; u < kU; ++u)
+                if (v0 + 32 * u < nvec) reinterpret_cast<VT*>(static_cast<T*>(dst) + off[u])[0] = val[u];
+        }
+    }
+}
+
+// ------------------------------------------------------------ wrapping tilers, 32-bit
+// Tilers whose pattern can leave the array (the paper's H/V input tilers wrap at the last repetition, Fig. 10
+// P:L681-687) with at most two wrapping array dims and all offsets < 2^31.  The flat offset is computed as if
+// nothing wrapped (one IMAD per combined dim, like the linear kernels) together with the raw coordinate of each
+// wrapping dim; the toroidal wrap is then one magic-number division per wrapping dim:
+//   (v mod s) * stride = v * stride - floor(v / s) * (s * stride).
+// Walked in tile order (tile side coalesced), all-32-bit, constants staged in shared memory.
+struct Wrap32Dev {
+    int32_t nd, nw;                                    // combined dims, wrapping array dims (0..2)
+    int32_t ext[2 * AOL_MAX_RANK], lin[2 * AOL_MAX_RANK];
+    uint32_t mul[2 * AOL_MAX_RANK], shift[2 * AOL_MAX_RANK];
+    int32_t wc[2][2 * AOL_MAX_RANK];                   // coefficient of combined dim d in wrapping dim k
+    int32_t worg[2], wext[2], wstep[2];                // origin, extent, extent * array stride
+    uint32_t wmul[2], wshift[2];
+    int32_t base, total;
+};
+
+template <int ES, int MODE>
+__global__ void __launch_bounds__(256) tiler_wrap32_kernel(const Wrap32Dev wd, const void* __restrict__ src,
+                                                           void* __restrict__ dst, unsigned long long* __restrict__ ws) {
+    using T = typename Elem<ES>::T;
+    __shared__ int4 pk[kND];   // {extent, magic multiplier, shift, flat-offset coefficient}
+    __shared__ int2 pw[kND];   // coefficients in the two wrapping dims
+    if (threadIdx.x < wd.nd) {
+        const int d = threadIdx.x;
+        pk[d] = make_int4(wd.ext[d], int32_t(wd.mul[d]), int32_t(wd.shift[d]), wd.lin[d]);
+        pw[d] = make_int2(wd.wc[0][d], wd.wc[1][d]);
+    }
+    __syncthreads();
+    const int32_t n_el = wd.total;
+    const int32_t stride = int32_t(gridDim.x * blockDim.x);
+    constexpr int kU = (MODE <= 1) ? 2 : 1;
+    const int32_t warp_first = int32_t((blockIdx.x * blockDim.x + (threadIdx.x & ~31u)) * kU + (threadIdx.x & 31u));
+    for (int32_t v0 = warp_first; v0 < n_el; v0 += kU * stride) {
+        int32_t off[kU], g[kU];
+#pragma unroll
+        for (int u = 0; u < kU; ++u) {
+            g[u] = v0 + 32 * u;
+            uint32_t n = g[u] < n_el ? uint32_t(g[u]) : 0u;
+            int32_t o = wd.base, w0 = wd.worg[0], w1 = wd.worg[1];
+#pragma unroll 1
+            for (int d = wd.nd - 1; d >= 0; --d) {
+                const int4 p = pk[d];
+                const int2 c = pw[d];
+                const uint32_t q = (__umulhi(n, uint32_t(p.y)) + n) >> p.z;
+                const int32_t i = int32_t(n - q * uint32_t(p.x));
+                n = q;
+                o += p.w * i;
+                w0 += c.x * i;
+                w1 += c.y * i;
+            }
+            if (wd.nw > 0) o -= int32_t((__umulhi(uint32_t(w0), wd.wmul[0]) + uint32_t(w0)) >> wd.wshift[0]) * wd.wstep[0];
+            if (wd.nw > 1) o -= int32_t((__umulhi(uint32_t(w1), wd.wmul[1]) + uint32_t(w1)) >> wd.wshift[1]) * wd.wstep[1];
+            off[u] = o;
+        }
+        if (MODE == 0) {   // gather: tiles[g] = array[off]
+            T val[kU];
+#pragma unroll
+            for (int u = 0; u < kU; ++u)
+                if (g[u] < n_el) val[u] = static_cast<const T*>(src)[off[u]];
+#pragma unroll
+            for (int u = 0; u < kU; ++u)
+                if (g[u] < n_el) static_cast<T*>(dst)[g[u]] = val[u];
+        } else if (MODE == 1) {   // FAST scatter: array[off] = tiles[g]
+            T val[kU];
+#pragma unroll
+            for (int u = 0; u < kU; ++u)
+                if (g[u] < n_el) val[u] = static_cast<const T*>(src)[g[u]];
+#pragma unroll
+            for (int u = 0; u < kU; ++u)
+                if (g[u] < n_el) static_cast<T*>(dst)[off[u]] = val[u];
+        } else if (MODE == 2) {   // SEQUENTIAL claim: the last (r, i) in row-major order wins
+            if (g[0] < n_el) atomicMax(ws + off[0], (unsigned long long)g[0] + 1ull);
+        } else {                  // SEQUENTIAL write
+            if (g[0] < n_el && ws[off[0]] == (unsigned long long)g[0] + 1ull)
+                static_cast<T*>(dst)[off[0]] = static_cast<const T*>(src)[g[0]];
+        }
+    }
+}
+
+// Fill *wd for a non-linear tiler if it qualifies (<= 2 wrapping dims, every unwrapped offset < 2^31).
+bool make_wrap32(const TilerDev& td, Wrap32Dev* wd) {
+    if (td.linear || !td.fast32 || td.array_elems >= (int64_t(1) << 31)) return false;
+    std::memset(wd, 0, sizeof *wd);
+    int wa[2], nw = 0;
+    for (int a = 0; a < td.ra; ++a)
+        if (!((td.nowrap_mask >> a) & 1)) {
+            if (nw == 2) return false;
+            wa[nw++] = a;
+        }
+    // the largest unwrapped flat offset: sum over array dims of (max raw coordinate) * stride
+    __int128 bound = 0;
+    for (int a = 0; a < td.ra; ++a) {
+        __int128 mx = td.org[a];
+        for (int d = 0; d < td.nd; ++d) mx += __int128(td.coef[a][d]) * (td.ext[d] - 1);
+        bound += mx * td.astride[a];
+    }
+    if (bound >= (__int128(1) << 31)) return false;
+    wd->nd = td.nd;
+    wd->nw = nw;
+    wd->total = int32_t(td.total);
+    int64_t base = 0;
+    for (int a = 0; a < td.ra; ++a) base += td.org[a] * td.astride[a];
+    wd->base = int32_t(base);
+    for (int d = 0; d < td.nd; ++d) {
+        int64_t l = 0;
+        for (int a = 0; a < td.ra; ++a) l += td.coef[a][d] * td.astride[a];
+        wd->ext[d] = int32_t(td.ext[d]);
+        wd->lin[d] = int32_t(l);
+        wd->mul[d] = td.fd_mul[d];
+        wd->shift[d] = td.fd_shift[d];
+        for (int k = 0; k < nw; ++k) wd->wc[k][d] = int32_t(td.coef[wa[k]][d]);
+    }
+    for (int k = 0; k < nw; ++k) {
+        const int a = wa[k];
+        const int64_t sa = td.ashape[a];
+        wd->worg[k] = int32_t(td.org[a]);
+        wd->wext[k] = int32_t(sa);
+        wd->wstep[k] = int32_t(sa * td.astride[a]);
+        uint32_t sh = 0;   // floor(v / s) == (umulhi(v, mul) + v) >> sh for v, s < 2^31
+        while (sh < 32 && (uint64_t(1) << sh) < uint64_t(sa)) ++sh;
+        wd->wmul[k] = uint32_t(((uint64_t(1) << 32) * ((uint64_t(1) << sh) - uint64_t(sa))) / uint64_t(sa) + 1);
+        wd->wshift[k] = sh;
+    }
+    return true;
+}
+
+// Gather / FAST scatter of the same tilers in blocks: the tile index space (natural order, tile side
+// contiguous) splits into INNER dims (the innermost ones, the outermost of them possibly in chunks) whose
+// product fills a block of <= kWTab elements, and OUTER dims enumerating the blocks.  Every block shares the
+// inner parts of the unwrapped flat offset and of the wrapping coordinates, so each CTA tabulates them once in
+// shared memory; an element then costs one LDS.128, three adds and the wrap fix-up instead of a digit-by-digit
+// decomposition (the per-element kernel above is issue/latency-bound on exactly that).
+constexpr int kWTab = 2048;   // 32 KB of int4 per CTA: 1024 entries 2.84 / 4096 2.61 / 2048 3.29 TB/s (wrapping d3)
+
+struct WrapTabDev {
+    int32_t n_in, n_out, nw;
+    int32_t in_ext[2 * AOL_MAX_RANK], in_lin[2 * AOL_MAX_RANK], in_w0[2 * AOL_MAX_RANK], in_w1[2 * AOL_MAX_RANK];
+    uint32_t in_mul[2 * AOL_MAX_RANK], in_shift[2 * AOL_MAX_RANK];
+    int32_t out_ext[2 * AOL_MAX_RANK + 1], out_lin[2 * AOL_MAX_RANK + 1], out_w0[2 * AOL_MAX_RANK + 1],
+        out_w1[2 * AOL_MAX_RANK + 1], out_g[2 * AOL_MAX_RANK + 1];
+    uint32_t out_mul[2 * AOL_MAX_RANK + 1], out_shift[2 * AOL_MAX_RANK + 1];
+    int32_t chunk_ext, chunk_len, inner, inner_tail, nblocks;
+    int32_t base, worg0, worg1, wext0, wext1, wstep0, wstep1;
+    uint32_t wmul0, wshift0, wmul1, wshift1;
+};
+
+template <int ES, int MODE>
+__global__ void __launch_bounds__(256) tiler_wraptab_kernel(const WrapTabDev wt, const void* __restrict__ src,
+                                                            void* __restrict__ dst) {
+    using T = typename Elem<ES>::T;
+    constexpr int kPer = kWTab / 256;
+    __shared__ int4 tab[kWTab];   // {flat offset, wrapping coordinate 0, wrapping coordinate 1} of the inner index
+    for (int e = threadIdx.x; e < wt.inner; e += 256) {
+        uint32_t n = uint32_t(e);
+        int32_t o = 0, w0 = 0, w1 = 0;
+        for (int d = wt.n_in - 1; d >= 0; --d) {
+            const uint32_t q = (__umulhi(n, wt.in_mul[d]) + n) >> wt.in_shift[d];
+            const int32_t i = int32_t(n - q * uint32_t(wt.in_ext[d]));
+            n = q;
+            o += wt.in_lin[d] * i;
+            w0 += wt.in_w0[d] * i;
+            w1 += wt.in_w1[d] * i;
+        }
+        tab[e] = make_int4(o, w0, w1, 0);
+    }
+    __syncthreads();
+    for (int32_t blk = blockIdx.x; blk < wt.nblocks; blk += gridDim.x) {
+        uint32_t n = uint32_t(blk);
+        int32_t bo = wt.base, b0 = wt.worg0, b1 = wt.worg1, bg = 0, count = wt.inner;
+        for (int d = wt.n_out - 1; d >= 0; --d) {
+            const uint32_t q = (__umulhi(n, wt.out_mul[d]) + n) >> wt.out_shift[d];
+            const int32_t i = int32_t(n - q * uint32_t(wt.out_ext[d]));
+            n = q;
+            bo += wt.out_lin[d] * i;
+            b0 += wt.out_w0[d] * i;
+            b1 += wt.out_w1[d] * i;
+            bg += wt.out_g[d] * i;
+            if (d == wt.n_out - 1)   // the chunk index: a partial last chunk holds fewer elements
+                count = min(wt.chunk_len, wt.chunk_ext - i * wt.chunk_len) * wt.inner_tail;
+        }
+        int32_t off[kPer];
+        T val[kPer];
+#pragma unroll
+        for (int k = 0; k < kPer; ++k) {
+            const int e = threadIdx.x + 256 * k;
+            const int4 t = tab[e < count ? e : 0];
+            int32_t o = bo + t.x;
+            const uint32_t w0 = uint32_t(b0 + t.y), w1 = uint32_t(b1 + t.z);
+            if (wt.nw > 0) o -= int32_t((__umulhi(w0, wt.wmul0) + w0) >> wt.wshift0) * wt.wstep0;
+            if (wt.nw > 1) o -= int32_t((__umulhi(w1, wt.wmul1) + w1) >> wt.wshift1) * wt.wstep1;
+            off[k] = o;
+        }
+#pragma unroll
+        for (int k = 0; k < kPer; ++k) {
+            const int e = threadIdx.x + 256 * k;
+            if (e < count) val[k] = MODE == 0 ? static_cast<const T*>(src)[off[k]] : static_cast<const T*>(src)[bg + e];
+        }
+#pragma unroll
+        for (int k = 0; k < kPer; ++k) {
+            const int e = threadIdx.x + 256 * k;
+            if (e < count) {
+                if (MODE == 0)
+                    static_cast<T*>(dst)[bg + e] = val[k];
+                else
+                    static_cast<T*>(dst)[off[k]] = val[k];
+            }
+        }
+    }
+}
+
+void magic32(int64_t ext, uint32_t* mul, uint32_t* shift) {
+    // n / ext == (umulhi(n, mul) + n) >> shift for n, ext < 2^31
+    uint32_t sh = 0;
+    while (sh < 32 && (uint64_t(1) << sh) < uint64_t(ext)) ++sh;
+    *mul = uint32_t(((uint64_t(1) << 32) * ((uint64_t(1) << sh) - uint64_t(ext))) / uint64_t(ext) + 1);
+    *shift = sh;
+}
+
+// Blocked form of a Wrap32Dev (natural tile order; tile strides from the extents).
+WrapTabDev make_wraptab(const Wrap32Dev& wd) {
+    WrapTabDev wt;
+    std::memset(&wt, 0, sizeof wt);
+    const int nd = wd.nd;
+    int64_t gst[2 * AOL_MAX_RANK];
+    int64_t g = 1;
+    for (int d = nd - 1; d >= 0; --d) {
+        gst[d] = g;
+        g *= wd.ext[d];
+    }
+    int k = nd - 1;
+    int64_t prod = 1;
+    while (k >= 0 && prod * wd.ext[k] <= kWTab) prod *= wd.ext[k--];
+    const int64_t c = k >= 0 ? std::max<int64_t>(1, kWTab / prod) : 1;
+    auto put_in = [&](int d, int64_t ext) {
+        wt.in_ext[wt.n_in] = int32_t(ext);
+        wt.in_lin[wt.n_in] = wd.lin[d];
+        wt.in_w0[wt.n_in] = wd.wc[0][d];
+        wt.in_w1[wt.n_in] = wd.wc[1][d];
+        magic32(ext, &wt.in_mul[wt.n_in], &wt.in_shift[wt.n_in]);
+        ++wt.n_in;
+    };
+    if (k >= 0) put_in(k, c);
+    for (int d = k + 1; d < nd; ++d) put_in(d, wd.ext[d]);
+    wt.inner = int32_t(prod * c);
+    wt.inner_tail = int32_t(prod);
+    wt.chunk_len = int32_t(c);
+    int64_t nblocks = 1;
+    auto put_out = [&](int64_t ext, int64_t lin, int64_t w0, int64_t w1, int64_t gs) {
+        wt.out_ext[wt.n_out] = int32_t(ext);
+        wt.out_lin[wt.n_out] = int32_t(lin);
+        wt.out_w0[wt.n_out] = int32_t(w0);
+        wt.out_w1[wt.n_out] = int32_t(w1);
+        wt.out_g[wt.n_out] = int32_t(gs);
+        magic32(ext, &wt.out_mul[wt.n_out], &wt.out_shift[wt.n_out]);
+        ++wt.n_out;
+        nblocks *= ext;
+    };
+    for (int d = 0; d < k; ++d) put_out(wd.ext[d], wd.lin[d], wd.wc[0][d], wd.wc[1][d], gst[d]);
+    const int64_t cext = k >= 0 ? wd.ext[k] : 1;
+    if (k >= 0)
+        put_out((cext + c - 1) / c, int64_t(wd.lin[k]) * c, int64_t(wd.wc[0][k]) * c, int64_t(wd.wc[1][k]) * c,
+                gst[k] * c);
+    else
+        put_out(1, 0, 0, 0, 0);
+    wt.chunk_ext = int32_t(cext);
+    wt.nblocks = int32_t(nblocks);
+    wt.base = wd.base;
+    wt.nw = wd.nw;
+    wt.worg0 = wd.worg[0];
+    wt.worg1 = wd.worg[1];
+    wt.wext0 = wd.wext[0];
+    wt.wext1 = wd.wext[1];
+    wt.wstep0 = wd.wstep[0];
+    wt.wstep1 = wd.wstep[1];
+    wt.wmul0 = wd.wmul[0];
+    wt.wshift0 = wd.wshift[0];
+    wt.wmul1 = wd.wmul[1];
+    wt.wshift1 = wd.wshift[1];
+    return wt;
+}
+
+// AOL_TILER_WRAPTAB=0 runs wrapping gathers / FAST scatters element by element (A/B measurements only).
+bool tiler_wraptab_enabled() {
+    static const bool v = [] {
+        const char* e = std::getenv("AOL_TILER_WRAPTAB");
+        return !(e && e[0] == '0');
+    }();
+    return v;
+}
+
+// AOL_TILER_WRAP32=0 keeps wrapping tilers on the 64-bit general kernel (A/B measurements only).
+bool tiler_wrap32_enabled() {
+    static const bool v = [] {
+        const char* e = std::getenv("AOL_TILER_WRAP32");
+        return !(e && e[0] == '0');
+    }();
+    return v;
+}
+
+int grid_for(int64_t n, int num_sms) {
+    return int(std::max<int64_t>(1, std::min<int64_t>((n + 255) / 256, int64_t(num_sms) * 32)));
+}
+
+template <int ES, int V, int MODE>
+aol_status_t launch_v(const TilerDev& td, const void* src, void* dst, unsigned long long* ws, int grid,
+                      cudaStream_t s) {
+    const bool fast = td.fast32 != 0, lin = td.linear != 0;
+    if (MODE <= 1 && lin && td.small32) {
+        DeviceInfo dev;
+        aol_status_t st = device_info(&dev);
+        if (st != AOL_OK) return st;
+        const int g32 = int(std::max<int64_t>(1, std::min<int64_t>((td.total / V + 255) / 256, int64_t(dev.num_sms) * 128)));
+        tiler_linear32_kernel<ES, V, MODE><<<g32, 256, 0, s>>>(td, src, dst);
+        AOL_LAUNCH_CHECK("tiler_linear32_kernel");
+        return AOL_OK;
+    }
+    if constexpr (V == 1) {
+        Wrap32Dev wd;
+        if (!lin && tiler_wrap32_enabled() && make_wrap32(td, &wd)) {
+            DeviceInfo dev;
+            aol_status_t st = device_info(&dev);
+            if (st != AOL_OK) return st;
+            if (MODE <= 1 && tiler_wraptab_enabled()) {
+                const WrapTabDev wt = make_wraptab(wd);
+                const int gt = int(std::max<int64_t>(1, std::min<int64_t>(wt.nblocks, int64_t(dev.num_sms) * 8)));
+                tiler_wraptab_kernel<ES, MODE><<<gt, 256, 0, s>>>(wt, src, dst);
+                AOL_LAUNCH_CHECK("tiler_wraptab_kernel");
+                return AOL_OK;
+            }
+            const int gw = int(std::max<int64_t>(1, std::min<int64_t>((td.total + 255) / 256, int64_t(dev.num_sms) * 128)));
+            tiler_wrap32_kernel<ES, MODE><<<gw, 256, 0, s>>>(wd, src, dst, ws);
+            AOL_LAUNCH_CHECK("tiler_wrap32_kernel");
+            return AOL_OK;
+        }
+    }
+    if (fast && lin)
+        tiler_kernel<ES, V, true, true, MODE><<<grid, 256, 0, s>>>(td, src, dst, ws);
+    else if (fast)
+        tiler_kernel<ES, V, true, false, MODE><<<grid, 256, 0, s>>>(td, src, dst, ws);
+    else if (lin)
+        tiler_kernel<ES, V, false, true, MODE><<<grid, 256, 0, s>>>(td, src, dst, ws);
+    else
+        tiler_kernel<ES, V, false, false, MODE><<<grid, 256, 0, s>>>(td, src, dst, ws);
+    AOL_LAUNCH_CHECK("tiler_kernel");
+    return AOL_OK;
+}
+
+template <int ES, int MODE>
+aol_status_t launch_es(const TilerDev& td, int vec, const void* src, void* dst, unsigned long long* ws,
+                       int num_sms, cudaStream_t s) {
+    const int grid = grid_for(td.total / vec, num_sms);
+    // vector width in elements (16, 8, 4 or 2 bytes) when the host proved contiguity + alignment, else 1
+    if (vec > 1) {
+        const int vb = ES * vec;
+        if constexpr (ES == 1) {
+            if (vb == 16) return launch_v<1, 16, MODE>(td, src, dst, ws, grid, s);
+            if (vb == 8) return launch_v<1, 8, MODE>(td, src, dst, ws, grid, s);
+            if (vb == 4) return launch_v<1, 4, MODE>(td, src, dst, ws, grid, s);
+            if (vb == 2) return launch_v<1, 2, MODE>(td, src, dst, ws, grid, s);
+        }
+        if constexpr (ES == 2) {
+            if (vb == 16) return launch_v<2, 8, MODE>(td, src, dst, ws, grid, s);
+            if (vb == 8) return launch_v<2, 4, MODE>(td, src, dst, ws, grid, s);
+            if (vb == 4) return launch_v<2, 2, MODE>(td, src, dst, ws, grid, s);
+        }
+        if constexpr (ES == 4) {
+            if (vb == 16) return launch_v<4, 4, MODE>(td, src, dst, ws, grid, s);
+            if (vb == 8) return launch_v<4, 2, MODE>(td, src, dst, ws, grid, s);
+        }
+        if constexpr (ES == 8) {
+            if (vb == 16) return launch_v<8, 2, MODE>(td, src, dst, ws, grid, s);
+        }
+    }
+    return launch_v<ES, 1, MODE>(td, src, dst, ws, grid_for(td.total, num_sms), s);
+}
+
+}  // namespace
+}  // namespace aol
