@@ -46,9 +46,24 @@ def _dtype_code(t: torch.Tensor) -> int:
     return _RAW[es]
 
 
-def _stream(stream: Optional[torch.cuda.Stream]) -> ctypes.c_void_p:
-    s = stream if stream is not None else torch.cuda.current_stream()
+def _stream(stream: Optional[torch.cuda.Stream], device=None) -> ctypes.c_void_p:
+    """The given stream, else the current stream of `device` (the tensors' device, not the current one)."""
+    s = stream if stream is not None else torch.cuda.current_stream(device)
     return ctypes.c_void_p(s.cuda_stream)
+
+
+def _out(t: torch.Tensor, shape, dtype, device, name: str) -> torch.Tensor:
+    """Check a caller-supplied output: the kernels write exactly `shape` elements of `dtype` on `device`."""
+    if tuple(t.shape) != tuple(shape) or t.dtype != dtype or t.device != device:
+        raise ValueError(f"{name} must be {dtype} {tuple(shape)} on {device}; got {t.dtype} {tuple(t.shape)} on "
+                         f"{t.device}")
+    return t
+
+
+def _checksum_buf(cs: torch.Tensor, n: int, device) -> torch.Tensor:
+    if cs.dtype not in (torch.uint64, torch.int64) or cs.numel() < n or cs.device != device:
+        raise ValueError(f"checksums must be a uint64/int64 tensor of >= {n} elements on {device}")
+    return cs
 
 
 def _dev(t: torch.Tensor, name: str) -> ctypes.c_void_p:
@@ -115,10 +130,10 @@ def tiler_gather(t: aol_tiler_t, array: torch.Tensor, out: Optional[torch.Tensor
         raise ValueError(f"array shape {tuple(array.shape)} != tiler array shape {arr}")
     if out is None:
         out = torch.empty(rep + pat, dtype=array.dtype, device=array.device)
-    elif tuple(out.shape) != rep + pat or out.dtype != array.dtype:
-        raise ValueError("out has the wrong shape or dtype")
-    check(lib().aol_tiler_gather(ctypes.byref(t), _dtype_code(array), _dev(array, "array"), _dev(out, "out"),
-                                 _stream(stream)))
+    _out(out, rep + pat, array.dtype, array.device, "out")
+    with torch.cuda.device(array.device):
+        check(lib().aol_tiler_gather(ctypes.byref(t), _dtype_code(array), _dev(array, "array"), _dev(out, "out"),
+                                     _stream(stream, array.device)))
     return out
 
 
@@ -126,17 +141,21 @@ def tiler_scatter(t: aol_tiler_t, tiles: torch.Tensor, array: torch.Tensor, mode
                   workspace: Optional[torch.Tensor] = None, stream: Optional[torch.cuda.Stream] = None) -> torch.Tensor:
     """array[(o + P.r + F.i) mod s] = tiles[r][i] in place (Fig. 6).  mode: 'fast' | 'sequential'."""
     arr, rep, pat = _shapes(t)
-    if tuple(array.shape) != arr or tuple(tiles.shape) != rep + pat or tiles.dtype != array.dtype:
-        raise ValueError("tiles/array shapes or dtypes do not match the tiler")
+    if tuple(array.shape) != arr:
+        raise ValueError(f"array shape {tuple(array.shape)} != tiler array shape {arr}")
+    _out(tiles, rep + pat, array.dtype, array.device, "tiles")
     m = {"fast": SCATTER_FAST, "sequential": SCATTER_SEQUENTIAL}[mode]
     ws_ptr, ws_bytes = ctypes.c_void_p(0), 0
     if m == SCATTER_SEQUENTIAL:
         need = int(lib().aol_tiler_scatter_workspace_bytes(ctypes.byref(t)))
         if workspace is None:
             workspace = torch.empty(need, dtype=torch.uint8, device=array.device)
+        if workspace.device != array.device:
+            raise ValueError("workspace must be on the array's device")
         ws_ptr, ws_bytes = _dev(workspace, "workspace"), workspace.numel() * workspace.element_size()
-    check(lib().aol_tiler_scatter(ctypes.byref(t), _dtype_code(array), _dev(tiles, "tiles"),
-                                  _dev(array, "array"), m, ws_ptr, ws_bytes, _stream(stream)))
+    with torch.cuda.device(array.device):
+        check(lib().aol_tiler_scatter(ctypes.byref(t), _dtype_code(array), _dev(tiles, "tiles"),
+                                      _dev(array, "array"), m, ws_ptr, ws_bytes, _stream(stream, array.device)))
     return array
 
 
@@ -173,7 +192,9 @@ def filter_apply(f: aol_filter_t, x: torch.Tensor, out: Optional[torch.Tensor] =
         raise ValueError(f"x must be int32 {a_in}")
     if out is None:
         out = torch.zeros(a_out, dtype=torch.int32, device=x.device)
-    check(lib().aol_filter_apply(ctypes.byref(f), _dev(x, "x"), _dev(out, "out"), _stream(stream)))
+    _out(out, a_out, torch.int32, x.device, "out")
+    with torch.cuda.device(x.device):
+        check(lib().aol_filter_apply(ctypes.byref(f), _dev(x, "x"), _dev(out, "out"), _stream(stream, x.device)))
     return out
 
 
@@ -197,7 +218,9 @@ def downscale_h(x: torch.Tensor, out: Optional[torch.Tensor] = None,
     planes, H, W = _planes(x)
     if out is None:
         out = torch.empty(x.shape[:-1] + (3 * (W // 8),), dtype=torch.int32, device=x.device)
-    check(lib().aol_downscale_h(_dev(x, "x"), _dev(out, "out"), planes, H, W, _stream(stream)))
+    _out(out, x.shape[:-1] + (3 * (W // 8),), torch.int32, x.device, "out")
+    with torch.cuda.device(x.device):
+        check(lib().aol_downscale_h(_dev(x, "x"), _dev(out, "out"), planes, H, W, _stream(stream, x.device)))
     return out
 
 
@@ -209,7 +232,9 @@ def downscale_v(y: torch.Tensor, out: Optional[torch.Tensor] = None,
     planes, H, W = _planes(y)
     if out is None:
         out = torch.empty(y.shape[:-2] + (4 * (H // 9), W), dtype=torch.int32, device=y.device)
-    check(lib().aol_downscale_v(_dev(y, "y"), _dev(out, "out"), planes, H, W, _stream(stream)))
+    _out(out, y.shape[:-2] + (4 * (H // 9), W), torch.int32, y.device, "out")
+    with torch.cuda.device(y.device):
+        check(lib().aol_downscale_v(_dev(y, "y"), _dev(out, "out"), planes, H, W, _stream(stream, y.device)))
     return out
 
 
@@ -239,13 +264,16 @@ def downscale_frame(x: torch.Tensor, out: Optional[torch.Tensor] = None, checksu
         raise TypeError("output must be int32 or int16")
     if out is None:
         out = torch.empty((N, C, 4 * (H // 9), 3 * (W // 8)), dtype=odt, device=x.device)
+    _out(out, (N, C, 4 * (H // 9), 3 * (W // 8)), odt, x.device, "out")
     cs = checksums
     if cs is True:
         cs = torch.empty(N, dtype=torch.uint64, device=x.device)
-    cs_ptr = _dev(cs, "checksums") if cs is not None else ctypes.c_void_p(0)
+    cs_ptr = _dev(_checksum_buf(cs, N, x.device), "checksums") if cs is not None else ctypes.c_void_p(0)
     o = _opts(opts)
-    check(lib().aol_downscale_frame_out(_dev(x, "x"), _TYPED[x.dtype], _dev(out, "out"), _TYPED[odt], N, C, H, W,
-                                        cs_ptr, ctypes.byref(o) if o is not None else None, _stream(stream)))
+    with torch.cuda.device(x.device):
+        check(lib().aol_downscale_frame_out(_dev(x, "x"), _TYPED[x.dtype], _dev(out, "out"), _TYPED[odt], N, C, H, W,
+                                            cs_ptr, ctypes.byref(o) if o is not None else None,
+                                            _stream(stream, x.device)))
     return out, cs
 
 
@@ -261,10 +289,14 @@ def downscale_frame_plan(frames: int, channels: int, H: int, W: int, dtype=torch
 def frame_checksum(z: torch.Tensor, out: Optional[torch.Tensor] = None,
                    stream: Optional[torch.cuda.Stream] = None) -> torch.Tensor:
     """Per-frame checksum of an int32 [frames][channels][Ho][Wo] batch."""
+    if z.dim() != 4 or z.dtype != torch.int32:
+        raise ValueError("z must be int32 [frames][channels][Ho][Wo]")
     N, C, Ho, Wo = z.shape
     if out is None:
         out = torch.empty(N, dtype=torch.uint64, device=z.device)
-    check(lib().aol_frame_checksum(_dev(z, "z"), N, C, Ho, Wo, _dev(out, "out"), _stream(stream)))
+    _checksum_buf(out, N, z.device)
+    with torch.cuda.device(z.device):
+        check(lib().aol_frame_checksum(_dev(z, "z"), N, C, Ho, Wo, _dev(out, "out"), _stream(stream, z.device)))
     return out
 
 
@@ -285,6 +317,9 @@ def downscale_frame_host(x: torch.Tensor, out: Optional[torch.Tensor] = None, ch
     device = torch.device(device if device is not None else "cuda")
     if out is None:
         out = torch.empty((N, C, 4 * (H // 9), 3 * (W // 8)), dtype=torch.int32, pin_memory=x.is_pinned())
+    _out(out, (N, C, 4 * (H // 9), 3 * (W // 8)), torch.int32, torch.device("cpu"), "out")
+    if not out.is_contiguous():
+        raise ValueError("out must be contiguous")
     cs = torch.empty(N, dtype=torch.uint64, pin_memory=x.is_pinned()) if checksums else None
     chunk = max(1, min(chunk_frames, N))
     need = host_workspace_bytes(chunk, C, H, W, x.dtype)
@@ -293,10 +328,11 @@ def downscale_frame_host(x: torch.Tensor, out: Optional[torch.Tensor] = None, ch
     if streams is None:
         streams = [torch.cuda.Stream(device=device) for _ in range(3)]
     sp = [ctypes.c_void_p(s.cuda_stream) for s in streams]
-    check(lib().aol_downscale_frame_host(
-        ctypes.c_void_p(x.data_ptr()), _TYPED[x.dtype], ctypes.c_void_p(out.data_ptr()), N, C, H, W,
-        ctypes.c_void_p(cs.data_ptr()) if cs is not None else ctypes.c_void_p(0), chunk,
-        _dev(workspace, "workspace"), workspace.numel(), sp[0], sp[1], sp[2]))
+    with torch.cuda.device(workspace.device):
+        check(lib().aol_downscale_frame_host(
+            ctypes.c_void_p(x.data_ptr()), _TYPED[x.dtype], ctypes.c_void_p(out.data_ptr()), N, C, H, W,
+            ctypes.c_void_p(cs.data_ptr()) if cs is not None else ctypes.c_void_p(0), chunk,
+            _dev(workspace, "workspace"), workspace.numel() * workspace.element_size(), sp[0], sp[1], sp[2]))
     return out, cs
 
 
@@ -307,6 +343,9 @@ def synth_frames(seed: int, frame0: int, nframes: int, channels: int, H: int, W:
     if out is None:
         out = torch.empty((nframes, channels, H, W), dtype=dtype,
                           device=device if device is not None else "cuda")
-    check(lib().aol_synth_frames(seed & 0xFFFFFFFFFFFFFFFF, frame0, nframes, channels, H, W, SYNTH_KINDS[kind],
-                                 value, _TYPED[out.dtype], _dev(out, "out"), _stream(stream)))
+    if out.numel() != nframes * channels * H * W or out.dtype not in (torch.int32, torch.uint8):
+        raise ValueError(f"out must hold {nframes}x{channels}x{H}x{W} int32 or uint8 elements")
+    with torch.cuda.device(out.device):
+        check(lib().aol_synth_frames(seed & 0xFFFFFFFFFFFFFFFF, frame0, nframes, channels, H, W, SYNTH_KINDS[kind],
+                                     value, _TYPED[out.dtype], _dev(out, "out"), _stream(stream, out.device)))
     return out

@@ -679,3 +679,31 @@ def test_concurrent_streams_and_threads(orc):
     for i in range(4):
         zo, cso = run_oracle(orc, inputs[i])
         assert np.array_equal(results[i][0], zo) and np.array_equal(results[i][1], cso)
+
+
+def test_binding_rejects_mismatched_buffers():
+    """The Python binding checks caller-supplied outputs before the C call: the kernels write exactly the
+    shape / dtype the ABI defines, so a smaller or differently typed buffer is refused (ValueError), never
+    overrun."""
+    x = aol.synth_frames(0, 0, 2, 3, 18, 64)
+    with pytest.raises(ValueError):
+        aol.downscale_frame(x, out=torch.empty((2, 3, 8, 23), dtype=torch.int32, device="cuda"))
+    with pytest.raises(TypeError):   # int64 is not an output type at all
+        aol.downscale_frame(x, out=torch.empty((2, 3, 8, 24), dtype=torch.int64, device="cuda"))
+    with pytest.raises(ValueError):
+        aol.downscale_frame(x, checksums=torch.empty(1, dtype=torch.uint64, device="cuda"))
+    with pytest.raises(ValueError):
+        aol.downscale_h(x, out=torch.empty((2, 3, 18, 23), dtype=torch.int32, device="cuda"))
+    with pytest.raises(ValueError):
+        aol.frame_checksum(x.to(torch.int64))
+    t = aol.make_tiler([16, 24], [2, 3], [8, 8], [0, 0], [[8, 0], [0, 8]], [[1, 0], [0, 1]])
+    A = torch.zeros((16, 24), dtype=torch.int32, device="cuda")
+    with pytest.raises(ValueError):
+        aol.tiler_gather(t, A, out=torch.empty((2, 3, 8, 7), dtype=torch.int32, device="cuda"))
+    with pytest.raises(ValueError):
+        aol.tiler_scatter(t, torch.zeros((2, 3, 8, 8), dtype=torch.int16, device="cuda"), A)
+    # the right buffers still work
+    z, cs = aol.downscale_frame(x, out=torch.empty((2, 3, 8, 24), dtype=torch.int32, device="cuda"),
+                                checksums=torch.empty(2, dtype=torch.int64, device="cuda"))
+    torch.cuda.synchronize()
+    assert z.shape == (2, 3, 8, 24)
