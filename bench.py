@@ -184,7 +184,7 @@ class ClockSampler:
                 "reasons": sorted(self.reasons), "samples": len(self.samples)}
 
 
-def cpu_baseline(a, gpu_cs=None, frame0=0, steps=1, min_seconds=0.0):
+def cpu_baseline(a, gpu_cs=None, frame0=0, steps=1, min_seconds=0.0, single_thread=False):
     """Time the CPU oracle (as it stands, OpenMP across planes) on a bounded sample.
     At least `steps` passes over the sample, and more until `min_seconds` of wall time
     have been spent (so the sample is ~10 s of work however many cores the host has).
@@ -217,7 +217,33 @@ def cpu_baseline(a, gpu_cs=None, frame0=0, steps=1, min_seconds=0.0):
                                         f"median pass of {len(times)} ({sum(times):.1f} s wall)", "seconds": dt}
     if gpu_cs is not None:
         info["parity_sample_ok"] = bool(np.array_equal(cs[:uniq], gpu_cs[:uniq]))
+    if single_thread:
+        # one frame on one thread, median of 3
+        st = []
+        for _ in range(3):
+            t0 = time.perf_counter()
+            oracle.downscale_frame(x[:1], nthreads=1)
+            st.append(time.perf_counter() - t0)
+        info["single_thread_s_per_frame"] = statistics.median(st)
+    info["host"] = host_cpu()
     return sample / dt, info
+
+
+def host_cpu():
+    """nproc, CPU model and socket count of the host the oracle ran on (from /proc/cpuinfo)."""
+    model, sockets = None, set()
+    try:
+        with open("/proc/cpuinfo") as f:
+            for line in f:
+                k, _, v = line.partition(":")
+                k, v = k.strip(), v.strip()
+                if k == "model name" and model is None:
+                    model = v
+                elif k == "physical id":
+                    sockets.add(v)
+    except OSError:
+        pass
+    return {"nproc": os.cpu_count(), "model": model, "sockets": len(sockets) or None}
 
 
 def run_reference(a, rank):
@@ -242,7 +268,7 @@ def run_reference(a, rank):
                    "channels": a.channels, "l2": "inputs larger than L2 (no flush)"},
         "impl": "reference",
         "cpu_baseline": {"value": value, "unit": "frames/s", "cores": info["cores"], "kind": "oracle",
-                         "sample": info["sample"]},
+                         "sample": info["sample"], "host": info.get("host")},
         "e2e": {"value": value, "unit": "frames/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
     }
     print(json.dumps(line), flush=True)
@@ -416,9 +442,11 @@ def main():
         line["gathered_checksums"] = int(cs_all.size)
     if world == 1 and not a.no_cpu_baseline:
         fps, info = cpu_baseline(a, gpu_cs=cs.cpu().view(torch.int64).numpy().view(np.uint64), frame0=frame0,
-                                 min_seconds=a.cpu_baseline_seconds)
+                                 min_seconds=a.cpu_baseline_seconds, single_thread=True)
         line["cpu_baseline"] = {"value": fps, "unit": "frames/s", "cores": info["cores"], "kind": "oracle",
-                                "sample": info["sample"], "parity_sample_ok": info.get("parity_sample_ok")}
+                                "sample": info["sample"], "parity_sample_ok": info.get("parity_sample_ok"),
+                                "single_thread_s_per_frame": info.get("single_thread_s_per_frame"),
+                                "host": info.get("host")}
     print(json.dumps(line), flush=True)
     if use_dist:
         dist.destroy_process_group()
