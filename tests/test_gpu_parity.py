@@ -707,3 +707,22 @@ def test_binding_rejects_mismatched_buffers():
                                 checksums=torch.empty(2, dtype=torch.int64, device="cuda"))
     torch.cuda.synchronize()
     assert z.shape == (2, 3, 8, 24)
+
+
+@pytest.mark.parametrize("dtype", [torch.uint8, torch.int32])
+def test_interleaved_to_planar_via_tiler(orc, dtype):
+    """SURVEY 8(f) f2's optional step: video frames arrive interleaved ([H][W][3], OpenCV's 24-bit BGR,
+    P:L260 / P:L657-659); the split into the planar [3][H][W] layout the filters take is itself an ArrayOL
+    tiler -- rep {3, H, W}, scalar pattern, paving mapping r = (c, y, x) to the array index (y, x, c).  The
+    generic gather does it; the result equals numpy's transpose and downscales to the oracle's output."""
+    H, W = 36, 64
+    xi = synth.frames(12, 0, 1, 1, H, W * 3, "uniform")[0, 0].reshape(H, W, 3)   # [H][W][3] samples 0..255
+    t = aol.make_tiler([H, W, 3], [3, H, W], [], [0, 0, 0], [[0, 1, 0], [0, 0, 1], [1, 0, 0]], [[], [], []])
+    planar = aol.tiler_gather(t, torch.from_numpy(xi.astype(np.uint8) if dtype == torch.uint8 else xi).cuda())
+    torch.cuda.synchronize()
+    ref = np.ascontiguousarray(np.transpose(xi, (2, 0, 1)))
+    assert np.array_equal(planar.cpu().numpy().astype(np.int32), ref)
+    z, cs = aol.downscale_frame(planar.unsqueeze(0), checksums=True)
+    zo, cso = orc.downscale_frame(ref[None].astype(np.int32))
+    torch.cuda.synchronize()
+    assert np.array_equal(z.cpu().numpy(), zo) and np.array_equal(np_u64(cs), cso)

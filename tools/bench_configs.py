@@ -193,6 +193,20 @@ def main():
               "check_wrap": bool(torch.equal(GH[0, 0, 239], torch.cat([X[0, 0, 1912:1920], X[0, 0, 0:3]])))})
         del X, GH
         torch.cuda.empty_cache()
+    if want("f2x"):
+        # f2's optional step: interleaved [N][H][W][3] 8-bit frames (OpenCV BGR) -> planar [N][3][H][W] as an
+        # ArrayOL tiler gather (rep {N, 3, H, W}, scalar pattern), 64 HD frames
+        N, H, W = 64, 1080, 1920
+        xi = torch.randint(0, 256, (N, H, W, 3), dtype=torch.uint8, device="cuda")
+        ti = aol.make_tiler([N, H, W, 3], [N, 3, H, W], [], [0, 0, 0, 0],
+                            [[1, 0, 0, 0], [0, 0, 1, 0], [0, 0, 0, 1], [0, 1, 0, 0]], [[], [], [], []])
+        xp = torch.empty((N, 3, H, W), dtype=torch.uint8, device="cuda")
+        tg, _ = timed(lambda: aol.tiler_gather(ti, xi, out=xp), inner=5)
+        emit({"config": "f2x interleaved -> planar split of 64 HD uint8 frames (tiler gather)", "ms": tg,
+              "GBps": 2 * xi.numel() / (tg / 1e3) / 1e9, "frames_per_s": N / (tg / 1e3),
+              "check": bool(torch.equal(xp[3, 1], xi[3, :, :, 1]))})
+        del xi, xp
+        torch.cuda.empty_cache()
     if want("f3"):
         # the paper's generic-vs-non-generic experiment on B200: run-time descriptors,
         # one fused gather+task+scatter kernel per filter, Y through HBM between the two filters
