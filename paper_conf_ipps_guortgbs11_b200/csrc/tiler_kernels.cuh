@@ -556,6 +556,223 @@ bool tiler_wrap32_enabled() {
     return v;
 }
 
+// ------------------------------------------------ deinterleave / interleave (linear tilers)
+// Linear tilers whose two innermost array-order dims are C (<= 8) interleaved channels of unit array stride
+// inside runs of X >= 64 positions that are contiguous on the TILE side, e.g. [N][H][W][3] video frames ->
+// [N][3][H][W] planes (SURVEY 8(f) f2's split, as a tiler gather) or back (the FAST scatter).  Element-wise
+// either the array side (stride-C reads) or the tile side (stride-S writes) is strided; here each CTA stages a
+// chunk of X positions x C channels in shared memory so both global sides are read / written contiguously.
+struct DeintDev {
+    int32_t n_out;                               // outer dims (array-order dims 0 .. nd-3)
+    int32_t out_ext[2 * AOL_MAX_RANK], out_lin[2 * AOL_MAX_RANK], out_gst[2 * AOL_MAX_RANK];
+    uint32_t out_mul[2 * AOL_MAX_RANK], out_shift[2 * AOL_MAX_RANK];
+    int32_t C, X, S;                             // channels, positions per run, tile stride of a channel
+    int32_t chunk, nchunks, nitems, base;        // positions per smem chunk, chunks per run, runs x chunks
+    uint32_t chunk_mul, chunk_shift;             // magic division by nchunks
+};
+
+constexpr int kDeintBytes = 16384;   // smem staging per CTA
+
+template <int ES, int MODE>
+__global__ void __launch_bounds__(256) tiler_deint_kernel(const DeintDev dd, const void* __restrict__ src,
+                                                          void* __restrict__ dst) {
+    using T = typename Elem<ES>::T;
+    constexpr int kV = 16 / ES;   // elements per 16-byte vector
+    __shared__ __align__(16) T buf[kDeintBytes / ES];
+    const int C = dd.C;
+    for (int32_t item = blockIdx.x; item < dd.nitems; item += gridDim.x) {
+        uint32_t n = uint32_t(item);
+        const uint32_t run = (__umulhi(n, dd.chunk_mul) + n) >> dd.chunk_shift;
+        const int32_t ck = int32_t(n - run * uint32_t(dd.nchunks));
+        n = run;
+        int32_t a0 = dd.base, t0 = 0;
+        for (int d = dd.n_out - 1; d >= 0; --d) {
+            const uint32_t q = (__umulhi(n, dd.out_mul[d]) + n) >> dd.out_shift[d];
+            const int32_t i = int32_t(n - q * uint32_t(dd.out_ext[d]));
+            n = q;
+            a0 += dd.out_lin[d] * i;
+            t0 += dd.out_gst[d] * i;
+        }
+        const int32_t x0 = ck * dd.chunk;
+        const int32_t nx = min(dd.chunk, dd.X - x0);
+        const int32_t ne = nx * C;
+        a0 += x0 * C;   // array: positions x0 .. x0+nx, all channels, contiguous
+        t0 += x0;       // tile: channel c run at t0 + c*S
+        // 16-byte vectors on a global side when its run starts 16-byte aligned and spans whole vectors
+        // (HD [N][H][W][3] bytes: always); element by element otherwise
+        const T* gsrc = static_cast<const T*>(src);
+        T* gdst = static_cast<T*>(dst);
+        const bool va = ((reinterpret_cast<uintptr_t>(MODE == 0 ? gsrc + a0 : gdst + a0)) & 15) == 0 && ne % kV == 0;
+        bool vt = nx % kV == 0 && (dd.S % kV) == 0;
+        vt = vt && ((reinterpret_cast<uintptr_t>(MODE == 0 ? gdst + t0 : gsrc + t0)) & 15) == 0;
+        if (MODE == 0) {
+            if (va) {
+                const uint4* A = reinterpret_cast<const uint4*>(gsrc + a0);
+                for (int32_t e = threadIdx.x; e < ne / kV; e += 256) reinterpret_cast<uint4*>(buf)[e] = A[e];
+            } else {
+                for (int32_t e = threadIdx.x; e < ne; e += 256) buf[e] = gsrc[a0 + e];
+            }
+            __syncthreads();
+            for (int c = 0; c < C; ++c) {
+                T* Tl = gdst + t0 + c * dd.S;
+                if (vt) {
+                    for (int32_t v = threadIdx.x; v < nx / kV; v += 256) {
+                        union { uint4 u; T e[kV]; } pk;
+#pragma unroll
+                        for (int j = 0; j < kV; ++j) pk.e[j] = buf[(v * kV + j) * C + c];
+                        reinterpret_cast<uint4*>(Tl)[v] = pk.u;
+                    }
+                } else {
+                    for (int32_t x = threadIdx.x; x < nx; x += 256) Tl[x] = buf[x * C + c];
+                }
+            }
+        } else {
+            for (int c = 0; c < C; ++c) {
+                const T* Tl = gsrc + t0 + c * dd.S;
+                if (vt) {
+                    for (int32_t v = threadIdx.x; v < nx / kV; v += 256) {
+                        union { uint4 u; T e[kV]; } pk;
+                        pk.u = reinterpret_cast<const uint4*>(Tl)[v];
+#pragma unroll
+                        for (int j = 0; j < kV; ++j) buf[(v * kV + j) * C + c] = pk.e[j];
+                    }
+                } else {
+                    for (int32_t x = threadIdx.x; x < nx; x += 256) buf[x * C + c] = Tl[x];
+                }
+            }
+            __syncthreads();
+            if (va) {
+                uint4* A = reinterpret_cast<uint4*>(gdst + a0);
+                for (int32_t e = threadIdx.x; e < ne / kV; e += 256) A[e] = reinterpret_cast<const uint4*>(buf)[e];
+            } else {
+                for (int32_t e = threadIdx.x; e < ne; e += 256) gdst[a0 + e] = buf[e];
+            }
+        }
+        __syncthreads();   // buf is reused by the next item
+    }
+}
+
+// The common video case of the above -- 3 interleaved 8-bit channels (24-bit RGB/BGR pixels), every
+// run 16-byte aligned on both sides -- needs no shared memory: a thread moves 16 pixels, three 16-byte loads of
+// packed pixels <-> one 16-byte vector per channel plane, the byte transpose done in registers with two PRMTs
+// per output word.  Lanes take consecutive 16-pixel groups, so both global sides stay coalesced.
+template <int kC>
+__device__ __forceinline__ uint32_t rgb_deint_word(uint32_t a, uint32_t b, uint32_t c) {
+    // bytes kC, kC+3, kC+6, kC+9 of the 12-byte window (a, b, c)
+    constexpr uint32_t o0 = kC, o1 = kC + 3, o2 = kC + 6, o3 = kC + 9;
+    constexpr uint32_t s1 = (o0 < 8 ? o0 : 0) | (o1 < 8 ? o1 : 0) << 4 | (o2 < 8 ? o2 : 0) << 8 | (o3 < 8 ? o3 : 0) << 12;
+    constexpr uint32_t s2 = (o0 < 8 ? 0u : o0 - 4) | (o1 < 8 ? 1u : o1 - 4) << 4 | (o2 < 8 ? 2u : o2 - 4) << 8 |
+                            (o3 < 8 ? 3u : o3 - 4) << 12;
+    return __byte_perm(__byte_perm(a, b, s1), c, s2);
+}
+
+// packed bytes 4k .. 4k+3 of a 12-byte group (4 pixels) from the three channel words p0, p1, p2
+template <int kK>
+__device__ __forceinline__ uint32_t rgb_int_word(uint32_t p0, uint32_t p1, uint32_t p2) {
+    // packed byte j = pixel (4kK + j) / 3, channel (4kK + j) % 3; first merge channels 0 and 1, then 2
+    constexpr int b0 = 4 * kK, b1 = b0 + 1, b2 = b0 + 2, b3 = b0 + 3;
+    constexpr uint32_t s1 = ((b0 % 3 == 2) ? 0u : uint32_t((b0 % 3) * 4 + b0 / 3)) |
+                            ((b1 % 3 == 2) ? 0u : uint32_t((b1 % 3) * 4 + b1 / 3)) << 4 |
+                            ((b2 % 3 == 2) ? 0u : uint32_t((b2 % 3) * 4 + b2 / 3)) << 8 |
+                            ((b3 % 3 == 2) ? 0u : uint32_t((b3 % 3) * 4 + b3 / 3)) << 12;
+    constexpr uint32_t s2 = ((b0 % 3 == 2) ? uint32_t(4 + b0 / 3) : 0u) | ((b1 % 3 == 2) ? uint32_t(4 + b1 / 3) : 1u) << 4 |
+                            ((b2 % 3 == 2) ? uint32_t(4 + b2 / 3) : 2u) << 8 | ((b3 % 3 == 2) ? uint32_t(4 + b3 / 3) : 3u) << 12;
+    return __byte_perm(__byte_perm(p0, p1, s1), p2, s2);
+}
+
+template <int MODE>
+__global__ void __launch_bounds__(256) tiler_rgb8_kernel(const DeintDev dd, const void* __restrict__ src,
+                                                         void* __restrict__ dst) {
+    const int32_t groups = dd.X / 16;   // 16-pixel groups per run
+    const int32_t total = dd.nitems;    // runs x groups
+    for (int32_t g = int32_t(blockIdx.x * blockDim.x + threadIdx.x); g < total; g += int32_t(gridDim.x * blockDim.x)) {
+        uint32_t n = uint32_t(g);
+        const uint32_t run = (__umulhi(n, dd.chunk_mul) + n) >> dd.chunk_shift;   // chunk_* = division by groups
+        const int32_t grp = int32_t(n - run * uint32_t(groups));
+        n = run;
+        int32_t a0 = dd.base, t0 = 0;
+        for (int d = dd.n_out - 1; d >= 0; --d) {
+            const uint32_t q = (__umulhi(n, dd.out_mul[d]) + n) >> dd.out_shift[d];
+            const int32_t i = int32_t(n - q * uint32_t(dd.out_ext[d]));
+            n = q;
+            a0 += dd.out_lin[d] * i;
+            t0 += dd.out_gst[d] * i;
+        }
+        a0 += 48 * grp;
+        t0 += 16 * grp;
+        if (MODE == 0) {
+            const uint4* A = reinterpret_cast<const uint4*>(static_cast<const uint8_t*>(src) + a0);
+            const uint4 u0 = A[0], u1 = A[1], u2 = A[2];
+            const uint32_t w[12] = {u0.x, u0.y, u0.z, u0.w, u1.x, u1.y, u1.z, u1.w, u2.x, u2.y, u2.z, u2.w};
+            uint8_t* T = static_cast<uint8_t*>(dst) + t0;
+            *reinterpret_cast<uint4*>(T) =
+                make_uint4(rgb_deint_word<0>(w[0], w[1], w[2]), rgb_deint_word<0>(w[3], w[4], w[5]),
+                           rgb_deint_word<0>(w[6], w[7], w[8]), rgb_deint_word<0>(w[9], w[10], w[11]));
+            *reinterpret_cast<uint4*>(T + dd.S) =
+                make_uint4(rgb_deint_word<1>(w[0], w[1], w[2]), rgb_deint_word<1>(w[3], w[4], w[5]),
+                           rgb_deint_word<1>(w[6], w[7], w[8]), rgb_deint_word<1>(w[9], w[10], w[11]));
+            *reinterpret_cast<uint4*>(T + 2 * dd.S) =
+                make_uint4(rgb_deint_word<2>(w[0], w[1], w[2]), rgb_deint_word<2>(w[3], w[4], w[5]),
+                           rgb_deint_word<2>(w[6], w[7], w[8]), rgb_deint_word<2>(w[9], w[10], w[11]));
+        } else {
+            const uint8_t* T = static_cast<const uint8_t*>(src) + t0;
+            const uint4 c0 = *reinterpret_cast<const uint4*>(T), c1 = *reinterpret_cast<const uint4*>(T + dd.S),
+                        c2 = *reinterpret_cast<const uint4*>(T + 2 * dd.S);
+            const uint32_t p0[4] = {c0.x, c0.y, c0.z, c0.w}, p1[4] = {c1.x, c1.y, c1.z, c1.w},
+                           p2[4] = {c2.x, c2.y, c2.z, c2.w};
+            uint32_t o[12];
+#pragma unroll
+            for (int q = 0; q < 4; ++q) {   // pixels 4q .. 4q+3 -> packed words 3q .. 3q+2
+                o[3 * q + 0] = rgb_int_word<0>(p0[q], p1[q], p2[q]);
+                o[3 * q + 1] = rgb_int_word<1>(p0[q], p1[q], p2[q]);
+                o[3 * q + 2] = rgb_int_word<2>(p0[q], p1[q], p2[q]);
+            }
+            uint4* A = reinterpret_cast<uint4*>(static_cast<uint8_t*>(dst) + a0);
+            A[0] = make_uint4(o[0], o[1], o[2], o[3]);
+            A[1] = make_uint4(o[4], o[5], o[6], o[7]);
+            A[2] = make_uint4(o[8], o[9], o[10], o[11]);
+        }
+    }
+}
+
+// AOL_TILER_DEINT=0 disables the staged (de)interleave kernel (A/B measurements only).
+bool tiler_deint_enabled() {
+    static const bool v = [] {
+        const char* e = std::getenv("AOL_TILER_DEINT");
+        return !(e && e[0] == '0');
+    }();
+    return v;
+}
+
+bool make_deint(const TilerDev& td, int es, DeintDev* dd) {
+    const int nd = td.nd;
+    if (!td.linear || !td.small32 || nd < 2) return false;
+    const int l = nd - 1, p = nd - 2;
+    if (td.p_lin[l] != 1 || td.p_ext[l] < 2 || td.p_ext[l] > 8) return false;
+    if (td.p_lin[p] != td.p_ext[l] || td.p_gst[p] != 1 || td.p_ext[p] < 64) return false;
+    if (td.p_gst[l] < td.p_ext[p]) return false;   // channel runs on the tile side must not interleave
+    std::memset(dd, 0, sizeof *dd);
+    dd->C = int32_t(td.p_ext[l]);
+    dd->X = int32_t(td.p_ext[p]);
+    dd->S = int32_t(td.p_gst[l]);
+    dd->chunk = std::max(32, (kDeintBytes / (dd->C * es)) & ~31);
+    dd->nchunks = (dd->X + dd->chunk - 1) / dd->chunk;
+    int64_t runs = 1;
+    for (int d = 0; d < p; ++d) {
+        dd->out_ext[d] = int32_t(td.p_ext[d]);
+        dd->out_lin[d] = int32_t(td.p_lin[d]);
+        dd->out_gst[d] = int32_t(td.p_gst[d]);
+        magic32(td.p_ext[d], &dd->out_mul[d], &dd->out_shift[d]);
+        runs *= td.p_ext[d];
+    }
+    dd->n_out = p;
+    magic32(dd->nchunks, &dd->chunk_mul, &dd->chunk_shift);
+    if (runs * dd->nchunks >= (int64_t(1) << 31)) return false;
+    dd->nitems = int32_t(runs * dd->nchunks);
+    dd->base = int32_t(td.base);
+    return true;
+}
+
 int grid_for(int64_t n, int num_sms) {
     return int(std::max<int64_t>(1, std::min<int64_t>((n + 255) / 256, int64_t(num_sms) * 32)));
 }
@@ -568,6 +785,30 @@ aol_status_t launch_v(const TilerDev& td, const void* src, void* dst, unsigned l
         DeviceInfo dev;
         aol_status_t st = device_info(&dev);
         if (st != AOL_OK) return st;
+        DeintDev dd;
+        if (V == 1 && tiler_deint_enabled() && make_deint(td, ES, &dd)) {
+            if constexpr (ES == 1) {
+                // 24-bit pixels with every run 16-byte aligned on both sides: the register transpose
+                const uintptr_t pa = reinterpret_cast<uintptr_t>(MODE == 0 ? src : dst);
+                const uintptr_t pt = reinterpret_cast<uintptr_t>(MODE == 0 ? dst : src);
+                bool ok = dd.C == 3 && dd.X % 16 == 0 && dd.S % 16 == 0 && dd.base % 16 == 0 && (pa | pt) % 16 == 0;
+                for (int d = 0; d < dd.n_out && ok; ++d) ok = dd.out_lin[d] % 16 == 0 && dd.out_gst[d] % 16 == 0;
+                const int64_t total = int64_t(dd.nitems / dd.nchunks) * (dd.X / 16);
+                if (ok && total < (int64_t(1) << 31)) {
+                    DeintDev rd = dd;
+                    rd.nitems = int32_t(total);
+                    magic32(dd.X / 16, &rd.chunk_mul, &rd.chunk_shift);
+                    const int gr = int(std::max<int64_t>(1, std::min<int64_t>((total + 255) / 256, int64_t(dev.num_sms) * 16)));
+                    tiler_rgb8_kernel<MODE><<<gr, 256, 0, s>>>(rd, src, dst);
+                    AOL_LAUNCH_CHECK("tiler_rgb8_kernel");
+                    return AOL_OK;
+                }
+            }
+            const int gd = int(std::max<int64_t>(1, std::min<int64_t>(dd.nitems, int64_t(dev.num_sms) * 8)));
+            tiler_deint_kernel<ES, MODE><<<gd, 256, 0, s>>>(dd, src, dst);
+            AOL_LAUNCH_CHECK("tiler_deint_kernel");
+            return AOL_OK;
+        }
         const int g32 = int(std::max<int64_t>(1, std::min<int64_t>((td.total / V + 255) / 256, int64_t(dev.num_sms) * 128)));
         tiler_linear32_kernel<ES, V, MODE><<<g32, 256, 0, s>>>(td, src, dst);
         AOL_LAUNCH_CHECK("tiler_linear32_kernel");

@@ -726,3 +726,26 @@ def test_interleaved_to_planar_via_tiler(orc, dtype):
     zo, cso = orc.downscale_frame(ref[None].astype(np.int32))
     torch.cuda.synchronize()
     assert np.array_equal(z.cpu().numpy(), zo) and np.array_equal(np_u64(cs), cso)
+
+
+@pytest.mark.parametrize("C,X,dtype", [(3, 64, np.uint8), (3, 1920, np.uint8), (2, 100, np.int16), (4, 5000, np.uint8),
+                                       (3, 6000, np.int32), (8, 70, np.int64), (3, 16385, np.uint8)])
+def test_deinterleave_tilers(orc, C, X, dtype):
+    """Linear tilers whose innermost array dims are C interleaved channels inside tile-contiguous runs of X
+    positions (the staged (de)interleave kernel; chunks of the run, ragged last chunk): gather == the C
+    oracle, FAST scatter inverts it."""
+    R = 3   # outer rows
+    arr, rep = [R, X, C], [C, R, X]
+    P = [[0, 1, 0], [0, 0, 1], [1, 0, 0]]
+    rng = np.random.default_rng(C * 1000 + X)
+    A = np.asarray(rng.integers(0, 100, size=arr)).astype(dtype)
+    ot = orc.make_tiler(arr, rep, [], [0, 0, 0], P, [[], [], []])
+    gt = aol.make_tiler(arr, rep, [], [0, 0, 0], P, [[], [], []])
+    Ad = torch.from_numpy(A).cuda()
+    G = aol.tiler_gather(gt, Ad)
+    torch.cuda.synchronize()
+    assert np.array_equal(G.cpu().numpy(), orc.gather(ot, A))
+    back = torch.zeros_like(Ad)
+    aol.tiler_scatter(gt, G, back, mode="fast")
+    torch.cuda.synchronize()
+    assert torch.equal(back, Ad)
