@@ -74,6 +74,15 @@ def main():
     G2 = aol.tiler_gather(tw, A[:9, :10].contiguous())
     C2 = torch.zeros((9, 10), dtype=torch.int32, device="cuda")
     aol.tiler_scatter(tw, G2, C2, mode="sequential")
+    # channel-interleaved runs: 3 x 8-bit (register transpose), 4 x 8-bit and 3 x 16-bit (smem-staged)
+    for C, X, dt in ((3, 64, torch.uint8), (4, 80, torch.uint8), (3, 96, torch.int16)):
+        ti = aol.make_tiler([2, X, C], [C, 2, X], [], [0, 0, 0], [[0, 1, 0], [0, 0, 1], [1, 0, 0]], [[], [], []])
+        Ai = (torch.arange(2 * X * C, device="cuda") % 97).to(dt).reshape(2, X, C)
+        Gi = aol.tiler_gather(ti, Ai)
+        ok &= torch.equal(Gi, Ai.permute(2, 0, 1))
+        Bi = torch.zeros_like(Ai)
+        aol.tiler_scatter(ti, Gi, Bi, mode="fast")
+        ok &= torch.equal(Ai, Bi)
     # a bijective blocking shifted to wrap in both dims (32-bit wrapping kernel): FAST scatter inverts the gather
     ts = aol.make_tiler([16, 24], [2, 3], [8, 8], [-3, 5], [[8, 0], [0, 8]], [[1, 0], [0, 1]])
     G3 = aol.tiler_gather(ts, A)
