@@ -20,4 +20,5 @@ timeout 900 ncu --set full --clock-control none --import-source on -k regex:fuse
 timeout 900 ncu --set full --clock-control none -k regex:tiler -s 1 -c 2 \
     -o gpurun_out/prof_tiler -f python tools/tiler_probe.py > gpurun_out/ncu_tiler.log 2>&1
 timeout 1500 python tools/bench_configs.py > gpurun_out/configs.jsonl 2> gpurun_out/configs.err
+timeout 300 python tools/bench_configs.py --only f2x >> gpurun_out/configs.jsonl 2>> gpurun_out/configs.err
 for f in 1 2; do timeout 600 python bench.py --dtype u8 --W 3840 --H 2160 --frames 64 --no-cpu-baseline --no-e2e >> gpurun_out/bench_u8_4k.jsonl 2>> gpurun_out/bench.err; done
