@@ -47,7 +47,8 @@ def parse():
     p.add_argument("--H", type=int, default=1080)
     p.add_argument("--W", type=int, default=1920)
     p.add_argument("--seed", type=int, default=0)
-    p.add_argument("--dtype", choices=["i32", "u8"], default="i32")
+    p.add_argument("--dtype", choices=["i32", "u8", "rgb8"], default="i32",
+                   help="input samples: int32 planes, uint8 planes, or packed 24-bit pixels [N][H][W][3]")
     p.add_argument("--out-dtype", choices=["i32", "i16"], default="i32",
                    help="output element type (i16 only with --dtype u8: NEXT row f1's int16 output option)")
     p.add_argument("--opts", type=str, default="", help='launch options JSON, e.g. {"ctas_per_sm":2}')
@@ -200,7 +201,7 @@ def cpu_baseline(a, gpu_cs=None, frame0=0, steps=1, min_seconds=0.0, single_thre
     sample = max(8, min(a.frames, 2 * nthreads))
     uniq = min(sample, 8)
     xu = synth.frames(a.seed, frame0, uniq, a.channels, a.H, a.W, "uniform")
-    if a.dtype == "u8":
+    if a.dtype in ("u8", "rgb8"):
         xu = xu.astype(np.int32)
     reps = (sample + uniq - 1) // uniq
     x = np.ascontiguousarray(np.concatenate([xu] * reps)[:sample])
@@ -322,17 +323,24 @@ def main():
     odtype = torch.int16 if a.out_dtype == "i16" else torch.int32
     if odtype == torch.int16 and tdtype != torch.uint8:
         raise SystemExit("--out-dtype i16 needs --dtype u8")
+    packed = a.dtype == "rgb8"
+    if packed and C != 3:
+        raise SystemExit("--dtype rgb8 (packed 24-bit pixels) needs --channels 3")
     x = aol.synth_frames(a.seed, frame0, F, C, H, W, "uniform", dtype=tdtype, device=dev)
+    if packed:   # the same frames as packed pixels [F][H][W][3] (built before timing)
+        x = x.permute(0, 2, 3, 1).contiguous()
+        a.no_e2e = True
     z = torch.empty((F, C, 4 * (H // 9), 3 * (W // 8)), dtype=odtype, device=dev)
     cs = torch.empty(F, dtype=torch.uint64, device=dev)
-    plan = aol.downscale_frame_plan(F, C, H, W, dtype=tdtype, opts=opts, out_dtype=odtype)
+    plan = aol.downscale_frame_plan(F, C, H, W, dtype="rgb8" if packed else tdtype, opts=opts, out_dtype=odtype)
     stream = torch.cuda.current_stream(dev)
+    run = aol.downscale_frame_packed if packed else aol.downscale_frame
 
     def step(record=None):
         for j, n in enumerate(calls):
             if record is not None:
                 record[0][j].record(stream)
-            aol.downscale_frame(x[:n], out=z[:n], checksums=cs[:n], opts=opts)
+            run(x[:n], out=z[:n], checksums=cs[:n], opts=opts)
             if record is not None:
                 record[1][j].record(stream)
 

@@ -63,7 +63,9 @@ typedef enum {
 
 typedef enum {
     AOL_U8 = 1, AOL_I16 = 2, AOL_I32 = 3, AOL_I64 = 4, /* typed elements            */
-    AOL_RAW8 = 5, AOL_RAW16 = 6, AOL_RAW32 = 7, AOL_RAW64 = 8 /* raw bytes, same sizes */
+    AOL_RAW8 = 5, AOL_RAW16 = 6, AOL_RAW32 = 7, AOL_RAW64 = 8, /* raw bytes, same sizes */
+    AOL_RGB8 = 9 /* fused downscaler input only: packed 24-bit pixels, frames [N][H][W][3] of 8-bit samples
+                    (P:L260's 24-bit RGB as OpenCV delivers it); channels must be 3 */
 } aol_dtype_t;
 
 typedef enum {
@@ -203,8 +205,9 @@ AOL_API aol_status_t aol_downscale_v(const int32_t* d_in, int32_t* d_out, int64_
  * never touches HBM -- the hand-written analogue of SaC's WITH-loop folding,
  * P:L528-546): d_in [frames][channels][H][W] -> d_out int32
  * [frames][channels][4H/9][3W/8], H filter first (Fig. 2).
- * in_dtype: AOL_I32 (values must lie in (-2^27, 2^27), reading Z12) or AOL_U8
- * (8-bit samples).  d_frame_checksums: nullable device u64 [frames],
+ * in_dtype: AOL_I32 (values must lie in (-2^27, 2^27), reading Z12), AOL_U8
+ * (8-bit samples) or AOL_RGB8 (packed pixels: d_in [frames][H][W][3] bytes, channels == 3,
+ * W % 16 == 0; the output is still planar).  d_frame_checksums: nullable device u64 [frames],
  * overwritten with  sum (u64)(u32)Z[n][c][y][x] * (1 + (c*Ho + y)*Wo + x)  mod 2^64.
  * frames == 0 is a no-op.  d_in/d_out 16-byte aligned.  Async on s. */
 AOL_API aol_status_t aol_downscale_frame(const void* d_in, aol_dtype_t in_dtype, int32_t* d_out, int64_t frames,

@@ -18,6 +18,7 @@ import torch
 
 from . import _lib
 from ._lib import FLAGS  # noqa: F401  (launch-option flag bits, include/aol.h AOL_FLAG_*)
+from ._lib import RGB8  # noqa: F401
 from ._lib import (FILTER_H, FILTER_V, AolError, I16, I32, I64, PRESET_H_IN, PRESET_H_OUT, PRESET_V_IN,
                    PRESET_V_OUT, RAW8, RAW16, RAW32, RAW64, SCATTER_FAST, SCATTER_SEQUENTIAL, U8, aol_filter_t,
                    aol_launch_opts_t, aol_plan_t, aol_tiler_t, check, lib)
@@ -25,7 +26,7 @@ from ._lib import (FILTER_H, FILTER_V, AolError, I16, I32, I64, PRESET_H_IN, PRE
 __all__ = [
     "AolError", "version", "make_tiler", "tiler_preset", "tiler_validate", "tiler_is_injective",
     "tiler_gather", "tiler_scatter", "downscale_h", "downscale_v", "downscale_frame", "downscale_frame_plan",
-    "frame_checksum", "downscale_frame_host", "synth_frames", "library_path",
+    "frame_checksum", "downscale_frame_host", "synth_frames", "library_path", "downscale_frame_packed",
     "PRESET_H_IN", "PRESET_H_OUT", "PRESET_V_IN", "PRESET_V_OUT", "SYNTH_KINDS",
     "make_filter", "filter_preset", "filter_validate", "filter_apply", "FILTER_H", "FILTER_V", "FLAGS",
 ]
@@ -277,11 +278,38 @@ def downscale_frame(x: torch.Tensor, out: Optional[torch.Tensor] = None, checksu
     return out, cs
 
 
+def downscale_frame_packed(x: torch.Tensor, out: Optional[torch.Tensor] = None, checksums=None, opts=None,
+                           stream: Optional[torch.cuda.Stream] = None, out_dtype: Optional[torch.dtype] = None):
+    """Fused downscaler on packed 24-bit pixels (OpenCV's interleaved frames): x uint8
+    [frames][H][W][3] -> planar [frames][3][4H/9][3W/8] int32 (or int16 with out_dtype=torch.int16).
+    Same integers and checksums as downscale_frame on the planar frames x.permute(0, 3, 1, 2)."""
+    if x.dim() != 4 or x.shape[3] != 3 or x.dtype != torch.uint8:
+        raise ValueError("x must be uint8 [frames][H][W][3]")
+    N, H, W, _ = x.shape
+    odt = out.dtype if out is not None else (out_dtype or torch.int32)
+    if odt not in (torch.int32, torch.int16):
+        raise TypeError("output must be int32 or int16")
+    if out is None:
+        out = torch.empty((N, 3, 4 * (H // 9), 3 * (W // 8)), dtype=odt, device=x.device)
+    _out(out, (N, 3, 4 * (H // 9), 3 * (W // 8)), odt, x.device, "out")
+    cs = checksums
+    if cs is True:
+        cs = torch.empty(N, dtype=torch.uint64, device=x.device)
+    cs_ptr = _dev(_checksum_buf(cs, N, x.device), "checksums") if cs is not None else ctypes.c_void_p(0)
+    o = _opts(opts)
+    with torch.cuda.device(x.device):
+        check(lib().aol_downscale_frame_out(_dev(x, "x"), RGB8, _dev(out, "out"), _TYPED[odt], N, 3, H, W, cs_ptr,
+                                            ctypes.byref(o) if o is not None else None, _stream(stream, x.device)))
+    return out, cs
+
+
 def downscale_frame_plan(frames: int, channels: int, H: int, W: int, dtype=torch.int32, opts=None,
                          out_dtype=torch.int32) -> dict:
+    """dtype: torch.int32 / torch.uint8 planes, or "rgb8" for packed 24-bit pixels."""
     p = aol_plan_t()
     o = _opts(opts)
-    check(lib().aol_downscale_frame_plan_out(_TYPED[dtype], _TYPED[out_dtype], frames, channels, H, W,
+    code = RGB8 if dtype == "rgb8" else _TYPED[dtype]
+    check(lib().aol_downscale_frame_plan_out(code, _TYPED[out_dtype], frames, channels, H, W,
                                              ctypes.byref(o) if o is not None else None, ctypes.byref(p)))
     return {f: getattr(p, f) for f, _ in aol_plan_t._fields_}
 

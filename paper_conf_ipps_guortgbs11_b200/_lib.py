@@ -21,6 +21,7 @@ STATUS_NAMES = {0: "AOL_OK", -1: "AOL_E_INVALID", -2: "AOL_E_SHAPE", -3: "AOL_E_
                 -5: "AOL_E_WORKSPACE", -6: "AOL_E_RANGE", -7: "AOL_E_CUDA"}
 # aol_dtype_t
 U8, I16, I32, I64, RAW8, RAW16, RAW32, RAW64 = 1, 2, 3, 4, 5, 6, 7, 8
+RGB8 = 9   # packed 24-bit pixels [frames][H][W][3] (fused downscaler input only)
 # aol_scatter_mode_t
 SCATTER_FAST, SCATTER_SEQUENTIAL = 0, 1
 # aol_preset_t

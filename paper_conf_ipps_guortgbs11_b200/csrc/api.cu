@@ -255,10 +255,13 @@ aol_status_t check_frame_args(const void* d_in, aol_dtype_t in_dtype, const void
                               int64_t channels, int64_t H, int64_t W, aol_dtype_t out_dtype = AOL_I32) {
     if (frames < 0 || channels <= 0 || H <= 0 || W <= 0)
         return fail(AOL_E_INVALID, "frames must be >= 0 and channels, H, W > 0");
-    if (in_dtype != AOL_I32 && in_dtype != AOL_U8) return fail(AOL_E_DTYPE, "in_dtype must be AOL_I32 or AOL_U8");
+    if (in_dtype != AOL_I32 && in_dtype != AOL_U8 && in_dtype != AOL_RGB8)
+        return fail(AOL_E_DTYPE, "in_dtype must be AOL_I32, AOL_U8 or AOL_RGB8");
     if (out_dtype != AOL_I32 && out_dtype != AOL_I16) return fail(AOL_E_DTYPE, "out_dtype must be AOL_I32 or AOL_I16");
-    if (out_dtype == AOL_I16 && in_dtype != AOL_U8)
-        return fail(AOL_E_DTYPE, "AOL_I16 output needs AOL_U8 input (8-bit samples give outputs in [-5, 255])");
+    if (out_dtype == AOL_I16 && in_dtype == AOL_I32)
+        return fail(AOL_E_DTYPE, "AOL_I16 output needs 8-bit input (8-bit samples give outputs in [-5, 255])");
+    if (in_dtype == AOL_RGB8 && channels != 3) return fail(AOL_E_SHAPE, "AOL_RGB8 (packed pixels) needs channels == 3");
+    if (in_dtype == AOL_RGB8 && W % 16) return fail(AOL_E_SHAPE, "AOL_RGB8 needs W % 16 == 0");
     if (W % 8) return fail(AOL_E_SHAPE, "W must be a multiple of 8 (H tiler paving step, Fig. 10)");
     if (H % 9) return fail(AOL_E_SHAPE, "H must be a multiple of 9 (V tiler paving step, reading Z1)");
     const __int128 in_elems = __int128(frames) * channels * H * W;
@@ -490,7 +493,7 @@ aol_status_t aol_frame_checksum(const int32_t* d_out, int64_t frames, int64_t ch
 
 size_t aol_downscale_frame_host_workspace_bytes(aol_dtype_t in_dtype, int64_t chunk_frames, int64_t channels,
                                                 int64_t H, int64_t W) {
-    const int es = in_dtype == AOL_U8 ? 1 : (in_dtype == AOL_I32 ? 4 : 0);
+    const int es = (in_dtype == AOL_U8 || in_dtype == AOL_RGB8) ? 1 : (in_dtype == AOL_I32 ? 4 : 0);
     if (!es || chunk_frames <= 0 || channels <= 0 || H <= 0 || W <= 0 || W % 8 || H % 9) return 0;
     const size_t in_b = (size_t(chunk_frames) * channels * H * W * es + 255) & ~size_t(255);
     const size_t out_b = (size_t(chunk_frames) * channels * (4 * (H / 9)) * (3 * (W / 8)) * 4 + 255) & ~size_t(255);
@@ -512,7 +515,7 @@ aol_status_t aol_downscale_frame_host(const void* h_in, aol_dtype_t in_dtype, in
     if (!d_workspace || ws_bytes < need) return fail(AOL_E_WORKSPACE, "device workspace too small");
     if (!aligned16(d_workspace)) return fail(AOL_E_ALIGN, "workspace must be 16-byte aligned");
 
-    const int es = in_dtype == AOL_U8 ? 1 : 4;
+    const int es = (in_dtype == AOL_U8 || in_dtype == AOL_RGB8) ? 1 : 4;
     const int64_t Ho = 4 * (H / 9), Wo = 3 * (W / 8);
     const size_t in_frame = size_t(channels) * H * W * es, out_frame = size_t(channels) * Ho * Wo * 4;
     const size_t in_b = (size_t(chunk_frames) * in_frame + 255) & ~size_t(255);

@@ -77,10 +77,12 @@ bool tma_shape_ok(aol_dtype_t dt, int64_t planes, int64_t channels, int64_t H, i
         return (layout == 128 ? W / 32 <= 256 : W / 8 <= 256) && planes * H < (int64_t(1) << 31);
     }
     if (dt == AOL_U8) return W % 16 == 0;   // 1-D bulk copies: 16-byte granularity
+    if (dt == AOL_RGB8) return W % 16 == 0;  // packed pixels: 9W-byte triples, 24-byte repetitions
     return false;
 }
 
 KernelFn pick(aol_dtype_t dt, int out_es, bool checksum, int kr, int64_t W, int flags, int block, int cps) {
+    if (dt == AOL_RGB8) return tma_kernel_rgb8(checksum, out_es == 2, block, cps);
     return dt == AOL_U8 ? tma_kernel_u8(checksum, out_es == 2, kr, block, cps)
                         : tma_kernel_i32(checksum, i32_layout(dt, W, flags), block, cps);
 }
@@ -103,11 +105,12 @@ struct RingGeom {
 
 RingGeom ring_geom(aol_dtype_t dt, int out_es, int64_t W, int flags) {
     // swizzled layouts need 1024-byte aligned stages (the swizzle atom); bulk copies 16 bytes (128 kept)
-    const uint32_t es = dt == AOL_U8 ? 1u : 4u, align = i32_layout(dt, W, flags) > 0 ? 1024u : 128u;
+    // bytes per input row: W int32 / W uint8 / 3W packed 24-bit pixels
+    const uint32_t es = dt == AOL_I32 ? 4u : (dt == AOL_RGB8 ? 3u : 1u), align = i32_layout(dt, W, flags) > 0 ? 1024u : 128u;
     RingGeom g;
     g.stage_bytes = uint32_t(rows_per_stage(dt, W, flags) * W) * es;
     g.stage_stride = (g.stage_bytes + align - 1) & ~(align - 1);
-    g.out_bytes = uint32_t(4 * out_es * (3 * (W / 8)));
+    g.out_bytes = uint32_t(4 * out_es * (3 * (W / 8))) * (dt == AOL_RGB8 ? 3u : 1u);   // packed: 3 planes
     return g;
 }
 
@@ -163,7 +166,9 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void*
     aol_status_t st = device_info(&dev);
     if (st != AOL_OK) return st;
     const aol_launch_opts_t o = opts ? *opts : aol_launch_opts_t{0, 0, 0, 0, 0};
-    const int64_t planes = frames * channels;
+    const bool rgb = in_dtype == AOL_RGB8;              // packed 24-bit pixels: a unit covers a frame's 3 planes
+    const bool u8like = in_dtype == AOL_U8 || rgb;     // 8-bit samples: issue-bound consumer
+    const int64_t planes = rgb ? frames : frames * channels;
     const int64_t Wo = 3 * (W / 8);
     *plan = FusedPlan{};
     plan->num_sms = dev.num_sms;
@@ -176,8 +181,8 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void*
     // repetitions per consumer thread: 2 for uint8 frames at least 1024 wide (HD: 0.498 vs 0.520 ms; 4K: equal),
     // 1 for narrower ones (CIF: 0.361 vs 0.315 ms -- one half-idle warp per CTA) and for int32
     // (profiles/r01_u8_r2_ab.jsonl)
-    const int kr = (in_dtype == AOL_U8 && W >= 1024 && !(o.flags & AOL_FLAG_U8_ONE_REP)) ? 2 : 1;
-    const int nc = int(((W / 8 / kr) + 31) / 32 * 32);
+    const int kr = rgb ? 3 : (in_dtype == AOL_U8 && W >= 1024 && !(o.flags & AOL_FLAG_U8_ONE_REP)) ? 2 : 1;
+    const int nc = int(((W / 8 / (rgb ? 1 : kr)) + 31) / 32 * 32);   // packed: one repetition (3 channels) per thread
     const int block = nc + 32;
     int stages = 0, cps = 1;
     if (tma_ok) {
@@ -189,7 +194,7 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void*
         // profiles/r01_u8_r2_ab.jsonl) -- 12 with int16 outputs, whose halved write traffic leaves DRAM room
         // for a third row stream per SM (HD: 0.431 ms at 3 CTAs/SM vs 0.503 at 2; profiles/r01_u8_i16.jsonl).
         const int cwarps = nc / 32;
-        const int want_warps = (in_dtype == AOL_U8 && kr == 1) ? 16 : (in_dtype == AOL_U8 && out_es == 2) ? 12 : 8;
+        const int want_warps = rgb ? 8 : (in_dtype == AOL_U8 && kr == 1) ? 16 : (in_dtype == AOL_U8 && out_es == 2) ? 12 : 8;
         cps = o.ctas_per_sm > 0 ? o.ctas_per_sm
                                 : std::max(1, std::min(8, (want_warps + cwarps - 1) / cwarps));
         for (;; --cps) {
@@ -224,6 +229,11 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void*
         return AOL_E_SHAPE;
     }
     if (o.kernel == 2) tma_ok = false;
+    if (rgb && !tma_ok) {
+        set_error("packed 24-bit pixels (AOL_RGB8) need the TMA fused kernel: W %% 16 == 0, W <= 7936, 16-byte "
+                  "aligned buffers");
+        return AOL_E_SHAPE;
+    }
 
     if (tma_ok) {
         const int nbands = int(H / 9);
@@ -238,7 +248,7 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void*
             // cheapest (largest on ties) wins (HD 0.479 ms at 20 bands vs 0.497 at 12, CIF 0.289 at 32 vs 0.310
             // at 8; profiles/r01_nb_sweep.jsonl).
             // (int16 outputs run 3 CTAs/SM: the epilogue weighs ~1.5x more; HD 0.421 ms at 20 vs 0.425 at 15)
-            const double ovh = in_dtype == AOL_U8 ? (out_es == 2 ? 5760.0 : 3840.0) / double(W) : 0.0;
+            const double ovh = u8like ? (out_es == 2 ? 5760.0 : 3840.0) / double(W) : 0.0;
             constexpr int kMaxNb = 120;
             const int max_nb = std::min(nbands, kMaxNb);
             double cost[kMaxNb + 1] = {};
@@ -250,7 +260,7 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void*
                 best = std::min(best, cost[cand]);
             }
             for (int cand = 1; cand <= max_nb; ++cand) {
-                if (in_dtype == AOL_U8) {
+                if (u8like) {
                     if (cost[cand] <= best) nb = cand;   // largest of the cheapest
                 } else if (cost[cand] <= 1.02 * best) {
                     nb = cand;                                   // smallest within 2 %
@@ -286,7 +296,8 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void*
 
 aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t in_dtype, void* d_out,
                           int64_t frames, int64_t channels, int64_t H, int64_t W, uint64_t* d_cs, cudaStream_t s) {
-    const int64_t planes = frames * channels;
+    const bool rgb = in_dtype == AOL_RGB8;
+    const int64_t planes = rgb ? frames : frames * channels;   // packed pixels: work units per frame
     const int32_t Ho = int32_t(4 * (H / 9)), Wo = int32_t(3 * (W / 8));
 
     if (plan.kernel == 2) {
@@ -331,7 +342,8 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
     a.W = int32_t(W);
     a.Ho = Ho;
     a.Wo = Wo;
-    a.channels = int32_t(channels);
+    a.channels = rgb ? 1 : int32_t(channels);   // packed: the unit index is the frame index
+    a.row_pitch = int32_t(rgb ? 3 * W : W);
     a.reps = int32_t(W / 8);
     a.segs = int32_t(layout == 32 ? W / 8 : W / 32);   // int32 swizzled lines per row (unused for linear rows)
     a.triples_per_plane = int32_t(H / 3);

@@ -18,6 +18,16 @@ KernelFn tma_kernel_u8h_nocs(int block, int cps);
 KernelFn tma_kernel_u8r2h_cs(int block, int cps);
 KernelFn tma_kernel_u8r2h_nocs(int block, int cps);
 
+KernelFn tma_kernel_rgb_cs(int block, int cps);
+KernelFn tma_kernel_rgb_nocs(int block, int cps);
+KernelFn tma_kernel_rgbh_cs(int block, int cps);
+KernelFn tma_kernel_rgbh_nocs(int block, int cps);
+
+KernelFn tma_kernel_rgb8(bool checksum, bool out16, int block, int cps) {
+    if (out16) return checksum ? tma_kernel_rgbh_cs(block, cps) : tma_kernel_rgbh_nocs(block, cps);
+    return checksum ? tma_kernel_rgb_cs(block, cps) : tma_kernel_rgb_nocs(block, cps);
+}
+
 KernelFn tma_kernel_i32(bool checksum, int layout, int block, int cps) {
     if (layout == 0) return checksum ? tma_kernel_i32l_cs(block, cps) : tma_kernel_i32l_nocs(block, cps);
     if (layout == 32) return checksum ? tma_kernel_i32s_cs(block, cps) : tma_kernel_i32s_nocs(block, cps);

@@ -83,6 +83,17 @@ __device__ __forceinline__ int32_t task_T_small(int32_t S) {
     return 7 * q - S;
 }
 
+// Packed 24-bit pixels (AOL_RGB8): bytes c, c+3, c+6, c+9 of the 12-byte window (a, b, c) -- channel kCh of
+// 4 consecutive pixels -- by two byte permutes.
+template <int kCh>
+__device__ __forceinline__ uint32_t rgb_channel_word(uint32_t a, uint32_t b, uint32_t c) {
+    constexpr uint32_t o0 = kCh, o1 = kCh + 3, o2 = kCh + 6, o3 = kCh + 9;
+    constexpr uint32_t s1 = (o0 < 8 ? o0 : 0) | (o1 < 8 ? o1 : 0) << 4 | (o2 < 8 ? o2 : 0) << 8 | (o3 < 8 ? o3 : 0) << 12;
+    constexpr uint32_t s2 = (o0 < 8 ? 0u : o0 - 4) | (o1 < 8 ? 1u : o1 - 4) << 4 | (o2 < 8 ? 2u : o2 - 4) << 8 |
+                            (o3 < 8 ? 3u : o3 - 4) << 12;
+    return __byte_perm(__byte_perm(a, b, s1), c, s2);
+}
+
 struct FusedArgs {
     void* Z;                    // output, Tout elements (int32, or int16 for 8-bit samples)
     uint64_t* cs;
@@ -107,6 +118,7 @@ struct FusedArgs {
     int32_t u8_tensor;      // uint8 path: 1 = 3-D TMA tensor loads (W % 128 == 0), 0 = 1-D bulk copies
     int32_t rows_per_stage; // int32 path: 3 (a stage holds a row triple) or 1 (one row per stage: finer ring
                             // granularity for wide frames); always 3 for uint8
+    int32_t row_pitch;      // uint8 paths: bytes per input row (W planar, 3W packed 24-bit pixels)
 };
 
 // Byte offset of 16-byte chunk `chunk` (0..7) of 128-byte line `line` under SWIZZLE_128B
@@ -183,6 +195,35 @@ __device__ __forceinline__ void h_row(uint32_t row_base, uint32_t rr, const RepG
         y[0] = task_T(e + qp);            // window cols 0..5
         y[1] = task_T(qp + f);            // window cols 2..7
         y[2] = task_T(q1.y + f + dn);     // window cols 5..10
+    } else if constexpr (kSwz == 3) {
+        // packed 24-bit pixels (kR = 3 channels of ONE repetition): the repetition's 8 pixels are 24 bytes at
+        // 24r, the next repetition's first 3 pixels 9 of the 12 bytes at 24(r+1) (0 for the row-wrapping one);
+        // each channel's samples are gathered into words by byte permutes, then summed like planar samples
+        static_assert(kR == 3, "packed pixels: 3 channels per thread");
+        const uint32_t rowa = row_base + rr * (3u * W);
+        const uint2 v0 = ptx::lds64(rowa + g.off0), v1 = ptx::lds64(rowa + g.off0 + 8u),
+                    v2 = ptx::lds64(rowa + g.off0 + 16u);
+        const uint2 n01 = ptx::lds64(rowa + g.offn);
+        const uint32_t n2 = ptx::lds32(rowa + g.offn + 8u);
+        uint32_t lo[3], hi[3], nw[3];
+        lo[0] = rgb_channel_word<0>(v0.x, v0.y, v1.x);
+        lo[1] = rgb_channel_word<1>(v0.x, v0.y, v1.x);
+        lo[2] = rgb_channel_word<2>(v0.x, v0.y, v1.x);
+        hi[0] = rgb_channel_word<0>(v1.y, v2.x, v2.y);
+        hi[1] = rgb_channel_word<1>(v1.y, v2.x, v2.y);
+        hi[2] = rgb_channel_word<2>(v1.y, v2.x, v2.y);
+        nw[0] = rgb_channel_word<0>(n01.x, n01.y, n2);
+        nw[1] = rgb_channel_word<1>(n01.x, n01.y, n2);
+        nw[2] = rgb_channel_word<2>(n01.x, n01.y, n2);
+#pragma unroll
+        for (int j = 0; j < 3; ++j) {
+            const int32_t S0 = int32_t(__dp4a(lo[j], 0x01010101u, __dp4a(hi[j], 0x00000101u, 0u)));
+            const int32_t S1 = int32_t(__dp4a(lo[j], 0x01010000u, __dp4a(hi[j], 0x01010101u, 0u)));
+            const int32_t S2 = int32_t(__dp4a(hi[j], 0x01010100u, __dp4a(nw[j], 0x00010101u, 0u)));
+            y[3 * j + 0] = task_T_nonneg(S0);
+            y[3 * j + 1] = task_T_nonneg(S1);
+            y[3 * j + 2] = task_T_nonneg(S2);
+        }
     } else {
         // uint8 samples: the kR repetitions' 8*kR bytes in 2*kR words, then the next repetition's first word
         // (columns 8(r+kR)..; word 0 for the row-wrapping repetition); dp4a(x, m, c) = c + sum of the bytes
@@ -225,7 +266,9 @@ template <typename Tin, typename Tout, int kR, int kSwz, bool kChecksum, int kMa
 __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
     fused_tma_kernel(const __grid_constant__ CUtensorMap tmap, const FusedArgs a) {
     constexpr bool kI32 = std::is_same<Tin, int32_t>::value;
-    constexpr int kC = 3 * kR;   // Y / Z columns per consumer thread
+    constexpr bool kIL = !kI32 && kSwz == 3;   // packed 24-bit pixels: a unit covers the 3 planes of a frame
+    constexpr int kC = 3 * kR;                 // Y / Z columns per consumer thread (kIL: 3 channels x 3)
+    constexpr int kRP = kIL ? 1 : kR;          // H-tiler repetitions per consumer thread
     extern __shared__ uint8_t smem_raw[];
     uint8_t* smem = reinterpret_cast<uint8_t*>((reinterpret_cast<uintptr_t>(smem_raw) + 1023) & ~uintptr_t(1023));
     uint8_t* stage_base = smem;
@@ -301,7 +344,7 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
                         // {128 B, W/128, rows} tensor, no swizzle: same linear smem layout as the bulk copy
                         ptx::tma_load_3d(dst, &tmap, &full[s], 0, 0, int32_t(row0 + 3 * trip));
                     } else {
-                        const uint8_t* src = static_cast<const uint8_t*>(a.X) + size_t(row0 + 3 * trip) * a.W;
+                        const uint8_t* src = static_cast<const uint8_t*>(a.X) + size_t(row0 + 3 * trip) * a.row_pitch;
                         ptx::bulk_load(dst, src, a.stage_bytes, &full[s]);
                     }
                     if (++s == a.stages) {
@@ -316,9 +359,9 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
 
     // ---------------------------------------------------- consumer threads
     const int lane = tid & 31;
-    const bool active = kR * tid < a.reps;
-    const int r = active ? kR * tid : a.reps - kR;   // first repetition owned (clamped for idle lanes)
-    const int rn = (r + kR == a.reps) ? 0 : r + kR;  // next thread's repetition (toroidal, Fig. 11 '% 1920')
+    const bool active = kRP * tid < a.reps;
+    const int r = active ? kRP * tid : a.reps - kRP;   // first repetition owned (clamped for idle lanes)
+    const int rn = (r + kRP == a.reps) ? 0 : r + kRP;  // next thread's repetition (toroidal, Fig. 11 '% 1920')
     RepGeom g;
     g.fix = (lane == 31) || (r + 1 == a.reps);
     g.swap = false;
@@ -338,6 +381,12 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
         g.off0 = (uint32_t(r) & 3u) << 1;   // chunk indices within the 128-byte line
         g.off1 = g.off0 + 1;
         g.offn = (uint32_t(rn) & 3u) << 1;
+    } else if constexpr (kIL) {
+        g.seg = g.segn = 0;
+        g.off0 = 24u * uint32_t(r);
+        g.off1 = g.off0 + 8;
+        g.offn = 24u * uint32_t(rn);
+        g.fix = false;
     } else {
         g.seg = g.segn = 0;
         g.off0 = 8u * uint32_t(r);
@@ -386,7 +435,24 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
             if (tid == 0) ptx::bulk_wait_read<kOutBufs - 1>();   // the out buffer we reuse is free again
             ptx::named_bar_sync(1, NC);
             const uint32_t ob = ptx::smem_u32(outbuf) + (emit_idx % kOutBufs) * a.out_bytes;
-            if (active) {
+            if constexpr (kIL) {
+              if (active) {
+                // packed pixels: channel j's 4 output rows are region j of the staging buffer (one plane each)
+#pragma unroll
+                for (int j = 0; j < 3; ++j)
+#pragma unroll
+                    for (int k = 0; k < 4; ++k) {
+                        const uint32_t e0 = uint32_t((4 * j + k) * Wo + 3 * r);
+#pragma unroll
+                        for (int m = 0; m < 3; ++m) {
+                            if constexpr (sizeof(Tout) == 4)
+                                ptx::sts32(ob + 4u * (e0 + m), z[k][3 * j + m]);
+                            else
+                                ptx::sts16(ob + 2u * (e0 + m), z[k][3 * j + m]);
+                        }
+                    }
+              }
+            } else if (active) {
 #pragma unroll
                 for (int k = 0; k < 4; ++k) {
                     const uint32_t e0 = uint32_t(k * Wo + 3 * r);   // element index of the thread's first column
@@ -409,7 +475,15 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
             }
             ptx::fence_proxy_async_smem();
             ptx::named_bar_sync(1, NC);
-            if (tid == 0) {
+            if (kIL && tid == 0) {   // one 4-row store per plane of the frame (kIL: compile-time)
+                const uint32_t pb = a.out_bytes / 3u;
+#pragma unroll
+                for (int j = 0; j < 3; ++j) {
+                    Tout* gz = static_cast<Tout*>(a.Z) + (size_t(3 * plane + j) * a.Ho + size_t(4 * band)) * size_t(Wo);
+                    ptx::bulk_store(gz, outbuf + (emit_idx % kOutBufs) * a.out_bytes + j * pb, pb);
+                }
+                ptx::bulk_commit();
+            } else if (tid == 0) {
                 Tout* gz = static_cast<Tout*>(a.Z) + (size_t(plane) * a.Ho + size_t(4 * band)) * size_t(Wo);
                 const uint8_t* src = outbuf + (emit_idx % kOutBufs) * a.out_bytes;
                 if (a.hint_stores)
@@ -419,7 +493,20 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
                 ptx::bulk_commit();
             }
             ++emit_idx;
-            if (kChecksum && active) {
+            if constexpr (kChecksum && kIL) {
+              if (active) {
+#pragma unroll
+                for (int j = 0; j < 3; ++j) {
+                    const uint32_t w0 = 1u + (uint32_t(j) * uint32_t(a.Ho) + uint32_t(4 * band)) * uint32_t(Wo) +
+                                        uint32_t(3 * r);
+#pragma unroll
+                    for (int k = 0; k < 4; ++k)
+#pragma unroll
+                        for (int m = 0; m < 3; ++m)
+                            csacc += uint64_t(uint32_t(z[k][3 * j + m])) * uint64_t(w0 + uint32_t(k * Wo + m));
+                }
+              }
+            } else if (kChecksum && active) {
                 // weight = 1 + frame-local flat index < 2^32 (the planner guarantees C*Ho*Wo < 2^32), so each
                 // term is one 32x32->64 multiply-add (IMAD.WIDE.U32 with a 64-bit addend)
                 const uint32_t w0 = 1u + (uint32_t(chan) * uint32_t(a.Ho) + uint32_t(4 * band)) * uint32_t(Wo) +
@@ -619,10 +706,15 @@ using KernelFn = void (*)(const CUtensorMap, const FusedArgs);
 // Explicit instantiations live in fused_k_*.cu (compiled in parallel); these pick one.
 KernelFn tma_kernel_i32(bool checksum, int layout, int block, int cps);   // layout = kSwz (128, 32 or 0)
 KernelFn tma_kernel_u8(bool checksum, bool out16, int reps_per_thread, int block, int cps);
+KernelFn tma_kernel_rgb8(bool checksum, bool out16, int block, int cps);   // packed 24-bit pixels
 
 template <typename Tin, typename Tout, int kR, int kSwz, bool kChecksum>
 KernelFn pick_tma_kernel(int block, int cps) {
-    if constexpr (kR == 2) {
+    if constexpr (kR == 3) {   // packed 24-bit pixels: 3 channels per thread
+        if (block <= 288 && cps >= 2) return fused_tma_kernel<Tin, Tout, kR, kSwz, kChecksum, 288, 2>;
+        if (block <= 512) return fused_tma_kernel<Tin, Tout, kR, kSwz, kChecksum, 512, 1>;
+        return fused_tma_kernel<Tin, Tout, kR, kSwz, kChecksum, 1024, 1>;
+    } else if constexpr (kR == 2) {
         // two repetitions per thread take ~126 registers: bounds that never force spills below 1024 threads
         if (block <= 160 && cps >= 3) return fused_tma_kernel<Tin, Tout, kR, kSwz, kChecksum, 160, 3>;
         if (block <= 256 && cps >= 2) return fused_tma_kernel<Tin, Tout, kR, kSwz, kChecksum, 256, 2>;

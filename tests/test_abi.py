@@ -255,7 +255,7 @@ def test_binding_constants_match_header():
     flags = {m.group(1): int(m.group(2)) for m in re.finditer(r"#define AOL_FLAG_(\w+)\s+(\d+)", hdr)}
     assert flags == aol.FLAGS
     for name, val in (("AOL_U8", _lib.U8), ("AOL_I16", _lib.I16), ("AOL_I32", _lib.I32), ("AOL_I64", _lib.I64),
-                      ("AOL_RAW8", _lib.RAW8), ("AOL_RAW64", _lib.RAW64), ("AOL_PRESET_V_OUT", _lib.PRESET_V_OUT),
+                      ("AOL_RAW8", _lib.RAW8), ("AOL_RAW64", _lib.RAW64), ("AOL_RGB8", _lib.RGB8), ("AOL_PRESET_V_OUT", _lib.PRESET_V_OUT),
                       ("AOL_SCATTER_SEQUENTIAL", _lib.SCATTER_SEQUENTIAL), ("AOL_FILTER_V", _lib.FILTER_V),
                       ("AOL_E_CUDA", -7)):
         m = re.search(name + r"\s*=\s*(-?\d+)", hdr)

@@ -749,3 +749,37 @@ def test_deinterleave_tilers(orc, C, X, dtype):
     aol.tiler_scatter(gt, G, back, mode="fast")
     torch.cuda.synchronize()
     assert torch.equal(back, Ad)
+
+
+@pytest.mark.parametrize("shape", [(2, 36, 128), (1, 9, 16), (3, 27, 352), (2, 18, 1040), (1, 1080, 1920),
+                                   (1, 18, 3840)])
+@pytest.mark.parametrize("out_dtype", [torch.int32, torch.int16])
+def test_packed_rgb_frames(orc, shape, out_dtype):
+    """Packed 24-bit pixels ([N][H][W][3], P:L260 as OpenCV delivers them) straight into the fused kernel
+    (AOL_RGB8: the consumer gathers each channel's samples with byte permutes): planar outputs and checksums
+    equal the oracle's on the transposed frames and the planar uint8 path's."""
+    N, H, W = shape
+    xp = synth.frames(21, 0, N, 3, H, W, "uniform")                      # planar int32 samples 0..255
+    packed = torch.from_numpy(np.ascontiguousarray(np.transpose(xp, (0, 2, 3, 1))).astype(np.uint8)).cuda()
+    zo, cso = run_oracle(orc, xp)
+    z, cs = aol.downscale_frame_packed(packed, checksums=True, out_dtype=out_dtype)
+    zp, csp = aol.downscale_frame(torch.from_numpy(xp.astype(np.uint8)).cuda(), checksums=True, out_dtype=out_dtype)
+    torch.cuda.synchronize()
+    assert np.array_equal(z.cpu().numpy().astype(np.int32), zo)
+    assert np.array_equal(np_u64(cs), cso)
+    assert torch.equal(z, zp) and torch.equal(cs.view(torch.int64), csp.view(torch.int64))
+    for opts in ({"bands_per_unit": 1, "stages": 2}, {"ctas_per_sm": 2}):
+        try:
+            z2, cs2 = aol.downscale_frame_packed(packed, checksums=True, out_dtype=out_dtype, opts=opts)
+        except aol.AolError:
+            # two CTAs of a 4K frame's 3-plane staging + 2 ring stages do not fit one SM's shared memory
+            assert W >= 3840 and opts.get("ctas_per_sm") == 2
+            continue
+        torch.cuda.synchronize()
+        assert torch.equal(z2, z) and np.array_equal(np_u64(cs2), cso), opts
+
+
+def test_packed_rgb_rejects():
+    x = torch.zeros((1, 18, 40, 3), dtype=torch.uint8, device="cuda")   # W % 16 != 0
+    with pytest.raises(aol.AolError):
+        aol.downscale_frame_packed(x)

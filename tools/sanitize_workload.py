@@ -48,6 +48,12 @@ def main():
                     ref = (z.clone(), cs.clone())
                 else:
                     ok &= torch.equal(z, ref[0]) and torch.equal(cs.view(torch.int64), ref[1].view(torch.int64))
+        if W % 16 == 0 and C == 3:   # packed 24-bit pixels into the fused kernel == the planar uint8 path
+            xu = aol.synth_frames(1, 0, N, C, H, W, "uniform", dtype=torch.uint8)
+            zp, csp = aol.downscale_frame_packed(xu.permute(0, 2, 3, 1).contiguous(), checksums=True)
+            zq, csq = aol.downscale_frame(xu, checksums=True)
+            torch.cuda.synchronize()
+            ok &= torch.equal(zp, zq) and torch.equal(csp.view(torch.int64), csq.view(torch.int64))
         if args.fused_only:
             continue
         x = aol.synth_frames(2, 0, N, C, H, W, "signed")
