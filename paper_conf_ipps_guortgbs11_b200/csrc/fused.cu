@@ -194,7 +194,9 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void*
         // profiles/r01_u8_r2_ab.jsonl) -- 12 with int16 outputs, whose halved write traffic leaves DRAM room
         // for a third row stream per SM (HD: 0.431 ms at 3 CTAs/SM vs 0.503 at 2; profiles/r01_u8_i16.jsonl).
         const int cwarps = nc / 32;
-        const int want_warps = rgb ? 8 : (in_dtype == AOL_U8 && kr == 1) ? 16 : (in_dtype == AOL_U8 && out_es == 2) ? 12 : 8;
+        // packed 24-bit pixels (3 channels per thread, ~100 registers): 16 warps (HD: 2 CTAs/SM 0.513 ms vs 0.608
+        // at 1; profiles/r01_rgb_sweep.jsonl)
+        const int want_warps = rgb ? 16 : (in_dtype == AOL_U8 && kr == 1) ? 16 : (in_dtype == AOL_U8 && out_es == 2) ? 12 : 8;
         cps = o.ctas_per_sm > 0 ? o.ctas_per_sm
                                 : std::max(1, std::min(8, (want_warps + cwarps - 1) / cwarps));
         for (;; --cps) {
