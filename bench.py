@@ -329,7 +329,6 @@ def main():
     x = aol.synth_frames(a.seed, frame0, F, C, H, W, "uniform", dtype=tdtype, device=dev)
     if packed:   # the same frames as packed pixels [F][H][W][3] (built before timing)
         x = x.permute(0, 2, 3, 1).contiguous()
-        a.no_e2e = True
     z = torch.empty((F, C, 4 * (H // 9), 3 * (W // 8)), dtype=odtype, device=dev)
     cs = torch.empty(F, dtype=torch.uint64, device=dev)
     plan = aol.downscale_frame_plan(F, C, H, W, dtype="rgb8" if packed else tdtype, opts=opts, out_dtype=odtype)
@@ -387,13 +386,14 @@ def main():
         chunk = 20
         ws = torch.empty(aol.host_workspace_bytes(chunk, C, H, W, tdtype), dtype=torch.uint8, device=dev)
         streams = [torch.cuda.Stream(device=dev) for _ in range(3)]
-        aol.downscale_frame_host(x_host, out=z_host, chunk_frames=chunk, workspace=ws, streams=streams, device=dev)
+        aol.downscale_frame_host(x_host, out=z_host, chunk_frames=chunk, workspace=ws, streams=streams, device=dev,
+                                 packed=packed)
         if use_dist:
             dist.barrier()
         t0 = time.perf_counter()
         for _ in range(a.e2e_steps):
             _, cs_h = aol.downscale_frame_host(x_host, out=z_host, chunk_frames=chunk, workspace=ws,
-                                               streams=streams, device=dev)
+                                               streams=streams, device=dev, packed=packed)
         e2e_s = time.perf_counter() - t0
         te = torch.tensor([e2e_s], dtype=torch.float64, device=dev if backend == "nccl" else "cpu")
         if use_dist:

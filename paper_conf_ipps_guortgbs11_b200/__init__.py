@@ -334,14 +334,20 @@ def host_workspace_bytes(chunk_frames: int, channels: int, H: int, W: int, dtype
 
 def downscale_frame_host(x: torch.Tensor, out: Optional[torch.Tensor] = None, checksums: bool = True,
                          chunk_frames: int = 16, workspace: Optional[torch.Tensor] = None, streams=None,
-                         device=None):
+                         device=None, packed: bool = False):
     """End-to-end from HOST memory (pinned for overlap): H2D, fused kernel, D2H, pipelined.
+    x: planar [N][C][H][W] int32 / uint8, or with packed=True uint8 [N][H][W][3] 24-bit pixels.
     Blocking.  Returns (out_host, checksums_host_or_None)."""
     if x.is_cuda:
         raise ValueError("x must be a host tensor")
     if not x.is_contiguous():
         raise ValueError("x must be contiguous")
-    N, C, H, W = x.shape
+    if packed:
+        if x.dim() != 4 or x.shape[3] != 3 or x.dtype != torch.uint8:
+            raise ValueError("packed x must be uint8 [frames][H][W][3]")
+        N, H, W, C = x.shape
+    else:
+        N, C, H, W = x.shape
     device = torch.device(device if device is not None else "cuda")
     if out is None:
         out = torch.empty((N, C, 4 * (H // 9), 3 * (W // 8)), dtype=torch.int32, pin_memory=x.is_pinned())
@@ -350,7 +356,8 @@ def downscale_frame_host(x: torch.Tensor, out: Optional[torch.Tensor] = None, ch
         raise ValueError("out must be contiguous")
     cs = torch.empty(N, dtype=torch.uint64, pin_memory=x.is_pinned()) if checksums else None
     chunk = max(1, min(chunk_frames, N))
-    need = host_workspace_bytes(chunk, C, H, W, x.dtype)
+    code = RGB8 if packed else _TYPED[x.dtype]
+    need = int(lib().aol_downscale_frame_host_workspace_bytes(code, chunk, C, H, W))
     if workspace is None:
         workspace = torch.empty(need, dtype=torch.uint8, device=device)
     if streams is None:
@@ -358,7 +365,7 @@ def downscale_frame_host(x: torch.Tensor, out: Optional[torch.Tensor] = None, ch
     sp = [ctypes.c_void_p(s.cuda_stream) for s in streams]
     with torch.cuda.device(workspace.device):
         check(lib().aol_downscale_frame_host(
-            ctypes.c_void_p(x.data_ptr()), _TYPED[x.dtype], ctypes.c_void_p(out.data_ptr()), N, C, H, W,
+            ctypes.c_void_p(x.data_ptr()), code, ctypes.c_void_p(out.data_ptr()), N, C, H, W,
             ctypes.c_void_p(cs.data_ptr()) if cs is not None else ctypes.c_void_p(0), chunk,
             _dev(workspace, "workspace"), workspace.numel() * workspace.element_size(), sp[0], sp[1], sp[2]))
     return out, cs

@@ -783,3 +783,15 @@ def test_packed_rgb_rejects():
     x = torch.zeros((1, 18, 40, 3), dtype=torch.uint8, device="cuda")   # W % 16 != 0
     with pytest.raises(aol.AolError):
         aol.downscale_frame_packed(x)
+
+
+def test_packed_rgb_host_streamed(orc):
+    """Packed 24-bit pixels from pinned HOST memory through the 3-stream pipeline (ragged last chunk):
+    outputs and checksums equal the device path's and the oracle's."""
+    N, H, W = 7, 36, 128
+    xp = synth.frames(23, 0, N, 3, H, W, "uniform")
+    packed = torch.from_numpy(np.ascontiguousarray(np.transpose(xp, (0, 2, 3, 1))).astype(np.uint8)).pin_memory()
+    z, cs = aol.downscale_frame_host(packed, chunk_frames=3, packed=True)
+    zo, cso = run_oracle(orc, xp)
+    assert np.array_equal(z.numpy(), zo)
+    assert np.array_equal(cs.view(torch.int64).numpy().view(np.uint64), cso)
