@@ -11,6 +11,7 @@ element written once.
   d4   64 frames of 3840x2160 (4K), same ratios
   f1   300 HD frames with uint8 samples
   f4   CIF 352x288, 2000 frames (Section III)
+  f1p  300 HD frames of packed 24-bit pixels (AOL_RGB8);  f2x interleaved -> planar split as a tiler gather
 """
 import argparse
 import json
@@ -241,6 +242,19 @@ def main():
         fused_line("f1 HD uint8 input, int16 output", 300, 3, 1080, 1920, dtype=torch.uint8, out_dtype=torch.int16)
     if want("f4"):
         fused_line("f4 CIF 2000 frames", 2000, 3, 288, 352)
+    if want("f1p"):
+        # packed 24-bit pixels [N][H][W][3] straight into the fused kernel (AOL_RGB8)
+        N, H, W = 300, 1080, 1920
+        xp = aol.synth_frames(3, 0, N, 3, H, W, dtype=torch.uint8).permute(0, 2, 3, 1).contiguous()
+        z = torch.empty((N, 3, 480, 720), dtype=torch.int32, device="cuda")
+        cs = torch.empty(N, dtype=torch.uint64, device="cuda")
+        med, mn = timed(lambda: aol.downscale_frame_packed(xp, out=z, checksums=cs), inner=5)
+        b = frames_bytes(N, 3, H, W, 1, 4)
+        emit({"config": "f1 HD packed 24-bit pixels (AOL_RGB8)", "shape": [N, H, W, 3], "timing": "5 calls back to back",
+              "ms": med, "min_ms": mn, "frames_per_s": N / (med / 1e3), "GBps": b / (med / 1e3) / 1e9,
+              "frac": b / (med / 1e3) / 1e9 / peak(), "plan": aol.downscale_frame_plan(N, 3, H, W, dtype="rgb8")})
+        del xp, z, cs
+        torch.cuda.empty_cache()
 
 
 if __name__ == "__main__":
