@@ -8,6 +8,7 @@ timeout 300 python -c "import __graft_entry__ as g; g.smoke()" > gpurun_out/smok
 timeout 600 python bench.py > gpurun_out/bench.json 2> gpurun_out/bench.err
 timeout 600 python bench.py --dtype u8 --no-cpu-baseline > gpurun_out/bench_u8.json 2>> gpurun_out/bench.err
 timeout 600 python bench.py --dtype u8 --out-dtype i16 --no-cpu-baseline > gpurun_out/bench_u8i16.json 2>> gpurun_out/bench.err
+timeout 600 python bench.py --dtype rgb8 --no-cpu-baseline > gpurun_out/bench_rgb8.json 2>> gpurun_out/bench.err
 timeout 600 python bench.py --impl reference --steps 2 --warmup 1 > gpurun_out/bench_reference.json 2>> gpurun_out/bench.err
 timeout 600 ncu --metrics gpu__time_duration.sum --clock-control none --csv --log-file gpurun_out/launches.csv \
     python bench.py --steps 3 --warmup 3 --no-e2e --no-cpu-baseline > gpurun_out/ncu_launch_bench.log 2>&1
@@ -20,5 +21,4 @@ timeout 900 ncu --set full --clock-control none --import-source on -k regex:fuse
 timeout 900 ncu --set full --clock-control none -k regex:tiler -s 1 -c 2 \
     -o gpurun_out/prof_tiler -f python tools/tiler_probe.py > gpurun_out/ncu_tiler.log 2>&1
 timeout 1500 python tools/bench_configs.py > gpurun_out/configs.jsonl 2> gpurun_out/configs.err
-timeout 300 python tools/bench_configs.py --only f2x >> gpurun_out/configs.jsonl 2>> gpurun_out/configs.err
 for f in 1 2; do timeout 600 python bench.py --dtype u8 --W 3840 --H 2160 --frames 64 --no-cpu-baseline --no-e2e >> gpurun_out/bench_u8_4k.jsonl 2>> gpurun_out/bench.err; done
