@@ -11,10 +11,11 @@ ARCH      := -gencode arch=compute_100a,code=sm_100a
 NVFLAGS   := $(ARCH) -O3 -lineinfo -std=c++17 -Xcompiler -fPIC,-fvisibility=hidden -Xptxas -v \
              --expt-relaxed-constexpr $(EXTRA)
 ORACLE    := oracle/liboracle.so
+SYNTH     := synth/libsynth.so
 
 EXAMPLE   := $(BUILD)/aol_example
 
-all: $(LIB) $(ORACLE) $(EXAMPLE)
+all: $(LIB) $(ORACLE) $(SYNTH) $(EXAMPLE)
 
 $(BUILD)/%.o: $(PKG)/csrc/%.cu $(CHDR)
 	@mkdir -p $(BUILD)
@@ -27,13 +28,17 @@ $(LIB): $(OBJS)
 # a plain-C client of the C ABI (no Python): examples/aol_example.c
 $(EXAMPLE): examples/aol_example.c include/aol.h $(LIB)
 	@mkdir -p $(BUILD)
-	gcc -std=c99 -O2 -Wall -Wextra -I include -I /usr/local/cuda/include $< -L $(PKG) -laol \
+	gcc -std=c11 -O2 -Wall -Wextra -I include -I /usr/local/cuda/include $< -L $(PKG) -laol \
 	    -L /usr/local/cuda/lib64 -lcudart -Wl,-rpath,'$$ORIGIN/../$(PKG)' -o $@
 
 $(ORACLE): oracle/aol_oracle.c oracle/aol_oracle.h
 	gcc -std=c99 -O2 -fopenmp -fPIC -shared -Wall -Wextra -o $@ oracle/aol_oracle.c
 
+# the seeded input generator in C (synth/synth.c; no method arithmetic): bench-size oracle inputs
+$(SYNTH): synth/synth.c
+	gcc -std=c99 -O2 -fopenmp -fPIC -shared -Wall -Wextra -o $@ synth/synth.c
+
 clean:
-	rm -rf $(BUILD) $(LIB) $(ORACLE)
+	rm -rf $(BUILD) $(LIB) $(ORACLE) $(SYNTH)
 
 .PHONY: all clean

@@ -5,22 +5,38 @@ Contract (driver): `python bench.py --gpus N --steps K --warmup W [--impl refere
 launched under torchrun for N > 1 (one process per GPU, NCCL).  Rank 0 prints
 ONE JSON line.
 
-Workload (BASELINE.json configs[1]): a 300-frame 1920x1080 3-channel synthetic
-int32 stream per GPU (weak scaling: each rank owns its own 300 frames, global
-frame indices rank*300 .. rank*300+299).  One step = one aol_downscale_frame
-call over the whole 300-frame batch, checksum epilogue included: every row of
-SURVEY.md 8(a) (a1-a9) runs inside the step.  Inputs (7.46 GB) are larger than
-the 126 MB L2, so no explicit flush is needed between steps.
+Headline workload (BASELINE.json configs[1]): a 300-frame
+1920x1080 3-channel synthetic int32 stream per GPU (weak scaling: each rank owns
+its own 300 frames, global frame indices rank*300 .. rank*300+299).  One step =
+one aol_downscale_frame call over the whole 300-frame batch, checksum epilogue
+included: every row of SURVEY.md 8(a) (a1-a9) runs inside the step.  Inputs
+(7.46 GB) are larger than the 126 MB L2, so no explicit flush is needed between
+steps.
 
 `value` is device-timed (CUDA events on the launching stream, barrier + sync on
 both sides, max over ranks); `e2e` is the same metric through the host-buffer
 C-ABI call (aol_downscale_frame_host: pinned H2D, kernel, D2H inside the timed
-region).  `cpu_baseline` times the CPU oracle (oracle/, test infrastructure)
-on a bounded sample of the same workload -- a reported baseline, not a target.
+region).
+
+Sub-records (`records`; --extras selects them) measure the other
+BASELINE.json configs in the same run, each with its roofline fraction and an
+in-run oracle parity flag: d1 (one HD frame: warm / cold-L2 / graph latency and
+host enqueue), d3 (generic tiler gather / FAST / SEQUENTIAL scatter on the
+SURVEY instance, a wrapping variant and the paper's H input tiler), d4 (64 4K
+frames), d5 (the 10,000-frame stream frame-sharded over the N ranks: strong
+scaling, at every N; every stream frame's checksum verified).
+
+The cpu_baseline leg (N = 1, rank 0) times the CPU oracle (oracle/, test
+infrastructure) over ALL 300 frames of the d2 workload, reports frames/s and
+algorithmic GB/s, and compares every frame's checksum with the GPU's; the same
+leg computes the oracle results behind the sub-records' parity flags.  It is a
+reported baseline, not a target.  `--impl reference` times the same oracle on
+the same workload as this tier's reference arm.
 """
 from __future__ import annotations
 
 import argparse
+import hashlib
 import json
 import os
 import statistics
@@ -34,9 +50,10 @@ if ROOT not in sys.path:
 
 METRIC = "HD->SD downscale frames/sec (1/2/4/8 B200) and achieved HBM GB/s vs peak"
 FALLBACK_HBM_GBS = 6650.0  # /opt/skills/guides/B200_PROFILING.md fallback
+ALL_EXTRAS = ("d1", "d3", "d4", "d5")
 
 
-def parse():
+def parse(argv=None):
     p = argparse.ArgumentParser()
     p.add_argument("--gpus", type=int, default=1)
     p.add_argument("--steps", type=int, default=100)
@@ -60,10 +77,33 @@ def parse():
     p.add_argument("--no-e2e", action="store_true")
     p.add_argument("--no-cpu-baseline", action="store_true")
     p.add_argument("--cpu-baseline-seconds", type=float, default=10.0,
-                   help="wall time the cpu_baseline leg spends re-running its sample (median pass reported)")
+                   help="oracle wall time the cpu_baseline leg spends re-running the workload (median pass)")
+    p.add_argument("--extras", type=str, default="auto",
+                   help="sub-records: comma list of d1,d3,d4,d5, 'all', 'none', or 'auto' (= all for the "
+                        "default int32 HD workload, none otherwise)")
+    p.add_argument("--d5-frames", type=int, default=10000)
+    p.add_argument("--d5-repeats", type=int, default=3)
+    p.add_argument("--ref-budget-seconds", type=float, default=240.0,
+                   help="--impl reference: bound on the whole run's oracle time (steps shrink to fit)")
     p.add_argument("--dump-checksums", type=str, default="",
                    help="rank 0 saves the gathered per-frame checksums (global frame order, .npy) for the tests")
-    return p.parse_args()
+    return p.parse_args(argv)
+
+
+def extras_of(a):
+    if a.extras == "auto":
+        default = (a.dtype == "i32" and a.out_dtype == "i32" and (a.H, a.W, a.channels) == (1080, 1920, 3)
+                   and not a.stream_frames and not a.opts)
+        return list(ALL_EXTRAS) if default else []
+    if a.extras in ("none", ""):
+        return []
+    if a.extras == "all":
+        return list(ALL_EXTRAS)
+    want = [e.strip() for e in a.extras.split(",") if e.strip()]
+    bad = [e for e in want if e not in ALL_EXTRAS]
+    if bad:
+        raise SystemExit(f"unknown --extras {bad}; choose from {ALL_EXTRAS}")
+    return want
 
 
 def workload_name(a):
@@ -73,11 +113,24 @@ def workload_name(a):
     return f"{a.frames}-frame {a.W}x{a.H} {a.channels}-channel synthetic stream per GPU, fused h+v downscale"
 
 
+def workload_config(a, world):
+    """The `config` object -- identical in the GPU arm and the reference arm (same workload)."""
+    return {"workload": workload_name(a), "frames_per_gpu": a.frames if not a.stream_frames else None,
+            "stream_frames": a.stream_frames or None, "H": a.H, "W": a.W, "channels": a.channels,
+            "in_dtype": a.dtype, "out_dtype": a.out_dtype, "seed": a.seed,
+            "l2": "inputs (7.46 GB at HD int32) larger than the 126 MB L2; no flush",
+            "parallelism": f"frame-sharded x{world} (no data-path collective)"}
+
+
 def bytes_per_frame(a):
     es = 4 if a.dtype == "i32" else 1
     eo = 2 if a.out_dtype == "i16" else 4
     Ho, Wo = 4 * (a.H // 9), 3 * (a.W // 8)
     return a.channels * (a.H * a.W * es + Ho * Wo * eo)
+
+
+def frame_bytes(C, H, W, es=4, eo=4):
+    return C * (H * W * es + (4 * (H // 9)) * (3 * (W // 8)) * eo)
 
 
 def measured_peak():
@@ -90,20 +143,49 @@ def measured_peak():
         return FALLBACK_HBM_GBS, "fallback (B200_PROFILING.md)"
 
 
-def ncu_traffic(a):
-    """(per-launch DRAM bytes, ncu DRAM utilisation in % of peak, capture tag) from the committed
-    `ncu --set full` summary, if it matches this workload; else (None, None, None)."""
+def src_hash():
+    """Hash of the CUDA library's sources (csrc/, include/, Makefile): an ncu capture is only quoted for the
+    tree it was taken on (tools/ncu_summary.py writes the same hash next to each capture)."""
+    h = hashlib.sha256()
+    files = []
+    for d in (os.path.join(ROOT, "paper_conf_ipps_guortgbs11_b200", "csrc"), os.path.join(ROOT, "include")):
+        for n in sorted(os.listdir(d)):
+            if n.endswith((".cu", ".cuh", ".h")):
+                files.append(os.path.join(d, n))
+    files.append(os.path.join(ROOT, "Makefile"))
+    for p in files:
+        h.update(os.path.relpath(p, ROOT).encode())
+        with open(p, "rb") as f:
+            h.update(f.read())
+    return h.hexdigest()[:16]
+
+
+def plan_key(plan):
+    return ",".join(f"{k}={plan[k]}" for k in ("kernel", "grid", "block", "smem_bytes", "stages", "bands_per_unit",
+                                                 "ctas_per_sm"))
+
+
+def traffic_key(a):
+    return f"{a.frames}x{a.channels}x{a.H}x{a.W}:{a.dtype}" + (":i16out" if a.out_dtype == "i16" else "")
+
+
+def ncu_traffic(a, plan):
+    """Per-launch DRAM bytes of the committed `ncu --set full` capture of THIS launch on THIS source tree:
+    (bytes, DRAM % of peak, capture tag, status).  The entry must match the workload, the hash of csrc/ and
+    the launch plan; otherwise bytes are None and status says why (a stale capture is never quoted)."""
     path = os.path.join(ROOT, "profiles", "ncu_traffic.json")
     try:
         with open(path) as f:
-            d = json.load(f)
-        key = f"{a.frames}x{a.channels}x{a.H}x{a.W}:{a.dtype}" + (":i16out" if a.out_dtype == "i16" else "")
-        e = d.get(key)
-        if e is None:
-            return None, None, None
-        return float(e["dram_bytes_per_launch"]), e.get("dram_pct_of_peak"), e.get("tag")
+            e = json.load(f).get(traffic_key(a))
     except Exception:
-        return None, None, None
+        e = None
+    if e is None:
+        return None, None, None, "no capture for this workload"
+    if e.get("src_hash") != src_hash():
+        return None, None, e.get("tag"), f"capture {e.get('tag')} is of another source tree"
+    if e.get("plan") != plan_key(plan):
+        return None, None, e.get("tag"), f"capture {e.get('tag')} used another launch plan"
+    return float(e["dram_bytes_per_launch"]), e.get("dram_pct_of_peak"), e.get("tag"), "same tree and plan"
 
 
 def mix_ceiling(a):
@@ -185,51 +267,6 @@ class ClockSampler:
                 "reasons": sorted(self.reasons), "samples": len(self.samples)}
 
 
-def cpu_baseline(a, gpu_cs=None, frame0=0, steps=1, min_seconds=0.0, single_thread=False):
-    """Time the CPU oracle (as it stands, OpenMP across planes) on a bounded sample.
-    At least `steps` passes over the sample, and more until `min_seconds` of wall time
-    have been spent (so the sample is ~10 s of work however many cores the host has).
-    Returns (frames_per_s, info): the median pass rate.  Also checks oracle checksums
-    against the GPU's for the unique sample frames when gpu_cs is given."""
-    import numpy as np
-
-    import oracle
-    import synth
-
-    cores = os.cpu_count() or 1
-    nthreads = max(1, min(cores, oracle.max_threads() if oracle.max_threads() > 0 else cores))
-    sample = max(8, min(a.frames, 2 * nthreads))
-    uniq = min(sample, 8)
-    xu = synth.frames(a.seed, frame0, uniq, a.channels, a.H, a.W, "uniform")
-    if a.dtype in ("u8", "rgb8"):
-        xu = xu.astype(np.int32)
-    reps = (sample + uniq - 1) // uniq
-    x = np.ascontiguousarray(np.concatenate([xu] * reps)[:sample])
-    oracle.downscale_frame(x[:1], nthreads=1)  # warm the library
-    times = []
-    cs = None
-    while len(times) < steps or sum(times) < min_seconds:
-        t0 = time.perf_counter()
-        _, cs = oracle.downscale_frame(x, nthreads=nthreads)
-        times.append(time.perf_counter() - t0)
-    dt = statistics.median(times)
-    info = {"cores": nthreads, "sample": f"{sample} frames of the workload ({uniq} unique, seed {a.seed}, "
-                                        f"frames {frame0}..{frame0 + uniq - 1} repeated), OpenMP over planes, "
-                                        f"median pass of {len(times)} ({sum(times):.1f} s wall)", "seconds": dt}
-    if gpu_cs is not None:
-        info["parity_sample_ok"] = bool(np.array_equal(cs[:uniq], gpu_cs[:uniq]))
-    if single_thread:
-        # SURVEY 8(d) (i): one frame on one thread, median of 3
-        st = []
-        for _ in range(3):
-            t0 = time.perf_counter()
-            oracle.downscale_frame(x[:1], nthreads=1)
-            st.append(time.perf_counter() - t0)
-        info["single_thread_s_per_frame"] = statistics.median(st)
-    info["host"] = host_cpu()
-    return sample / dt, info
-
-
 def host_cpu():
     """nproc, CPU model and socket count of the host the oracle ran on (from /proc/cpuinfo)."""
     model, sockets = None, set()
@@ -247,33 +284,403 @@ def host_cpu():
     return {"nproc": os.cpu_count(), "model": model, "sockets": len(sockets) or None}
 
 
-def run_reference(a, rank):
-    """--impl reference: the CPU oracle is this tier's reference arm (rank 0 only)."""
+# ============================================================ cpu_baseline leg (the CPU oracle)
+# The only code in bench.py (besides --impl reference, which calls it) that runs oracle/.  Inputs come from the
+# seeded generator synth/ (its C/OpenMP form, untimed); only the oracle calls are timed.
+
+def oracle_threads():
+    import oracle
+
+    cores = os.cpu_count() or 1
+    mt = oracle.max_threads()
+    return max(1, min(cores, mt if mt > 0 else cores))
+
+
+def oracle_checksums(seed, index, C, H, W, nthreads, chunk=None):
+    """Oracle per-frame checksums of the synthetic frames whose global indices are `index` (in order), in chunks
+    of frames.  Returns (u64 checksums, seconds spent inside the oracle)."""
+    import numpy as np
+
+    import oracle
+    import synth
+
+    index = list(index)
+    chunk = chunk or max(1, min(32, nthreads))
+    xbuf = np.empty((min(chunk, max(1, len(index))), C, H, W), dtype=np.int32)
+    out = np.empty(len(index), dtype=np.uint64)
+    spent = 0.0
+    for k in range(0, len(index), chunk):
+        idx = index[k:k + chunk]
+        x = xbuf[:len(idx)]
+        synth.frames_c(seed, 0, len(idx), C, H, W, "uniform", index=idx, out=x, nthreads=nthreads)
+        t0 = time.perf_counter()
+        _, cs = oracle.downscale_frame(x, nthreads=nthreads)
+        spent += time.perf_counter() - t0
+        out[k:k + len(idx)] = cs
+    return out, spent
+
+
+def cpu_baseline(a, frame0, nframes, gpu_cs=None, min_seconds=0.0, single_thread=False):
+    """the oracle (as it stands, OpenMP across planes, -O2) over EVERY frame of the workload,
+    passes repeated until `min_seconds` of oracle time; the median pass gives frames/s and algorithmic GB/s.
+    The first pass's checksums are compared with the GPU's for every frame (parity_all_frames)."""
+    import numpy as np
+
+    nthreads = oracle_threads()
+    index = list(range(frame0, frame0 + nframes))
+    passes, cs0 = [], None
+    while not passes or sum(passes) < min_seconds:
+        cs, spent = oracle_checksums(a.seed, index, a.channels, a.H, a.W, nthreads)
+        passes.append(spent)
+        if cs0 is None:
+            cs0 = cs
+    dt = statistics.median(passes)
+    fps = nframes / dt
+    rec = {"value": fps, "unit": "frames/s", "cores": nthreads, "kind": "oracle",
+           "sample": (f"all {nframes} frames of the workload (seed {a.seed}, global frames {frame0}..{frame0 + nframes - 1}), "
+                      f"OpenMP over planes, median of {len(passes)} passes ({sum(passes):.1f} s of oracle time; "
+                      f"input generation untimed)"),
+           "GBps_algorithmic": frame_bytes(a.channels, a.H, a.W) * fps / 1e9, "seconds_per_pass": dt,
+           "frames": nframes, "host": host_cpu(), "label": "CPU oracle, not a competitor"}
+    if gpu_cs is not None:
+        rec["parity_all_frames"] = bool(np.array_equal(cs0, gpu_cs))
+        rec["frames_compared"] = int(min(len(cs0), len(gpu_cs)))
+        if not rec["parity_all_frames"]:
+            rec["mismatched_frames"] = [int(i) for i in np.nonzero(cs0 != gpu_cs)[0][:16]]
+    if single_thread:
+        # SURVEY 8(d) (i): one frame on one thread, median of 3
+        import oracle
+        import synth
+
+        x1 = synth.frames_c(a.seed, frame0, 1, a.channels, a.H, a.W)
+        st = []
+        for _ in range(3):
+            t0 = time.perf_counter()
+            oracle.downscale_frame(x1, nthreads=1)
+            st.append(time.perf_counter() - t0)
+        rec["single_thread_s_per_frame"] = statistics.median(st)
+        rec["single_thread_GBps_algorithmic"] = frame_bytes(a.channels, a.H, a.W) / rec["single_thread_s_per_frame"] / 1e9
+    return rec
+
+
+def cpu_parity_frame(seed, frame0, C, H, W, z_dev, cs_dev):
+    """d1: the whole output array and checksum of one frame against the oracle."""
+    import numpy as np
+
+    import oracle
+    import synth
+
+    zo, cso = oracle.downscale_frame(synth.frames_c(seed, frame0, 1, C, H, W), nthreads=oracle_threads())
+    return bool(np.array_equal(z_dev, zo) and np.array_equal(cs_dev, cso))
+
+
+def cpu_parity_tiler(arr, rep, pat, origin, paving, fitting, A_pre, G_pre=None, B_pre=None, mode=None):
+    """d3: a prefix of the tiler's leading (repetition = array) dimension computed by the oracle: the gathered
+    tiles G_pre, or the array B_pre after scattering G_pre into zeros (mode 'fast' / 'sequential' share the
+    oracle's Fig. 6 loop)."""
+    import numpy as np
+
+    import oracle
+
+    t = oracle.make_tiler(arr, rep, pat, origin, paving, fitting)
+    G = oracle.gather(t, A_pre)
+    if mode is None:
+        return bool(np.array_equal(G, G_pre))
+    return bool(np.array_equal(oracle.scatter(t, G_pre, np.zeros_like(A_pre)), B_pre))
+
+
+# ============================================================ GPU timing helpers
+
+def timed(fn, reps=20, warm=3, before=None, inner=1):
+    """Median and min ms per call (CUDA events on the current stream, after warm-up); `inner` calls back to back
+    between the events (for sub-millisecond kernels, where one call per event pair times the launch gap)."""
+    import torch
+
+    s = torch.cuda.current_stream()
+    for _ in range(warm):
+        if before:
+            before()
+        fn()
+    torch.cuda.synchronize()
+    ts = []
+    for _ in range(reps):
+        if before:
+            before()
+        e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        e0.record(s)
+        for _ in range(inner):
+            fn()
+        e1.record(s)
+        torch.cuda.synchronize()
+        ts.append(e0.elapsed_time(e1) / inner)
+    return statistics.median(ts), min(ts)
+
+
+# ============================================================ sub-records (SURVEY 8(d) d1, d3, d4, d5)
+
+def record_d1(aol, peak, check):
+    """configs[0]: one HD frame -- latency, not bandwidth (29 MB fits in L2)."""
+    import numpy as np
+    import torch
+
+    N, C, H, W, seed = 1, 3, 1080, 1920, 0
+    x = aol.synth_frames(seed, 0, N, C, H, W)
+    z = torch.empty((N, C, 480, 720), dtype=torch.int32, device="cuda")
+    cs = torch.empty(N, dtype=torch.uint64, device="cuda")
+    call = lambda: aol.downscale_frame(x, out=z, checksums=cs)  # noqa: E731
+    # warm L2: a GPU-side sleep before each call keeps the host enqueue off the device timeline
+    warm, _ = timed(call, reps=50, before=lambda: torch.cuda._sleep(200000))
+    flush = torch.empty(512 << 20, dtype=torch.uint8, device="cuda")   # > 2x the 126 MB L2
+    cold, _ = timed(call, reps=50, before=lambda: flush.fill_(1))
+    del flush
+    torch.cuda.synchronize()
+    t0 = time.perf_counter()
+    for _ in range(200):
+        call()
+    host_us = (time.perf_counter() - t0) / 200 * 1e6
+    torch.cuda.synchronize()
+    # device time per call with the host removed: 20 calls captured in a CUDA graph, replayed
+    g = torch.cuda.CUDAGraph()
+    s = torch.cuda.Stream()
+    s.wait_stream(torch.cuda.current_stream())
+    with torch.cuda.stream(s):
+        call()
+        torch.cuda.synchronize()
+        with torch.cuda.graph(g, stream=s):
+            for _ in range(20):
+                call()
+    torch.cuda.synchronize()
+    graph_ms, _ = timed(lambda: g.replay(), reps=20)
+    b = frame_bytes(C, H, W)
+    rec = {"config": "d1 single 1920x1080 3-channel frame -> 720x480 (BASELINE configs[0])",
+           "warm_l2_us": warm * 1e3, "cold_l2_us": cold * 1e3, "graph_us_per_call": graph_ms * 1e3 / 20,
+           "host_enqueue_us_per_call_python": host_us, "roofline_floor_us": b / peak / 1e3,
+           "frac_cold": (b / peak / 1e3) / (cold * 1e3), "frac_graph": (b / peak / 1e3) / (graph_ms * 1e3 / 20),
+           "timing": "CUDA events, median of 50 (warm: 200 us GPU sleep before each call; cold: 512 MB fill before "
+                     "each call); graph: 20 calls per replay, median of 20",
+           "plan": aol.downscale_frame_plan(N, C, H, W)}
+    torch.cuda.synchronize()
+    rec["_parity_args"] = (seed, 0, C, H, W, z.cpu().numpy(), cs.cpu().view(torch.int64).numpy().view(np.uint64))
+    if check:
+        rec["parity"] = cpu_parity_frame(*rec["_parity_args"])
+    del rec["_parity_args"]
+    return rec
+
+
+def record_d3(aol, peak, check):
+    """configs[2]: generic tiler gather / scatter on SURVEY 8(d) d3's perf instance ({64,1024,1024} int32 -> 8x8
+    tiles), the same blocking wrapping toroidally in both image dims, and the paper's H input tiler (Fig. 10,
+    wraps at the last repetition) over 64 HD planes.  Algorithmic bytes: tiles written (read) + distinct array
+    elements read (written)."""
+    import torch
+
+    out = []
+    arr, rep, pat = [64, 1024, 1024], [64, 128, 128], [8, 8]
+    P, F = [[1, 0, 0], [0, 8, 0], [0, 0, 8]], [[0, 0], [1, 0], [0, 1]]
+    A = torch.randint(0, 1 << 30, tuple(arr), dtype=torch.int32, device="cuda")
+    G = torch.empty(tuple(rep + pat), dtype=torch.int32, device="cuda")
+    B = torch.zeros_like(A)
+    ws = torch.empty(int(aol.tiler_scatter_workspace_bytes(aol.make_tiler(arr, rep, pat, [0, 0, 0], P, F))),
+                     dtype=torch.uint8, device="cuda")
+    nb = 2 * A.numel() * 4
+    pre = 2   # oracle parity on the first `pre` slices of dim 0 (a repetition dim with paving 1: a sub-tiler)
+    for name, origin in (("blocking 8x8 (SURVEY d3 perf instance)", [0, 0, 0]),
+                         ("blocking 8x8 wrapping in both image dims (origin (0,-3,5))", [0, -3, 5])):
+        t = aol.make_tiler(arr, rep, pat, origin, P, F)
+        tg, _ = timed(lambda: aol.tiler_gather(t, A, out=G), inner=10)
+        B.zero_()
+        tf, _ = timed(lambda: aol.tiler_scatter(t, G, B, mode="fast"), inner=10)
+        roundtrip = bool(torch.equal(A, B))
+        B.zero_()
+        tq, _ = timed(lambda: aol.tiler_scatter(t, G, B, mode="sequential", workspace=ws), inner=5)
+        roundtrip_seq = bool(torch.equal(A, B))
+        rec = {"config": f"d3 generic tiler {name}: array {arr} int32, rep {rep}, pattern {pat}",
+               "gather_ms": tg, "gather_GBps": nb / tg / 1e6, "gather_frac": nb / tg / 1e6 / peak,
+               "scatter_fast_ms": tf, "scatter_fast_GBps": nb / tf / 1e6, "scatter_fast_frac": nb / tf / 1e6 / peak,
+               "scatter_seq_ms": tq, "scatter_seq_GBps": nb / tq / 1e6, "scatter_seq_frac": nb / tq / 1e6 / peak,
+               "algorithmic_bytes_per_call": nb, "timing": "CUDA events, 10 (SEQUENTIAL: 5) calls back to back per "
+               "event pair, median of 20",
+               "roundtrip_gather_scatter_identity": roundtrip and roundtrip_seq}
+        if check:
+            sub = ([pre] + arr[1:], [pre] + rep[1:])
+            Ap = A[:pre].cpu().numpy()
+            Gp = G[:pre].cpu().numpy()
+            rec["parity"] = (cpu_parity_tiler(sub[0], sub[1], pat, origin, P, F, Ap, G_pre=Gp)
+                             and cpu_parity_tiler(sub[0], sub[1], pat, origin, P, F, Ap, G_pre=Gp,
+                                                  B_pre=B[:pre].cpu().numpy(), mode="sequential")
+                             and rec["roundtrip_gather_scatter_identity"])
+            rec["parity_scope"] = (f"oracle on slices 0..{pre - 1} of 64 (gather and SEQUENTIAL scatter); gather -> "
+                                   "scatter identity on the whole array (FAST and SEQUENTIAL)")
+        out.append(rec)
+    del A, G, B, ws
+    torch.cuda.empty_cache()
+    # the paper's H input tiler over 64 HD planes (array {64,1080,1920}, rep {64,1080,240}, pattern {11})
+    X = aol.synth_frames(0, 0, 64, 1, 1080, 1920).reshape(64, 1080, 1920)
+    arr, rep, pat = [64, 1080, 1920], [64, 1080, 240], [11]
+    P, F = [[1, 0, 0], [0, 1, 0], [0, 0, 8]], [[0], [0], [1]]
+    th = aol.make_tiler(arr, rep, pat, [0, 0, 0], P, F)
+    GH = torch.empty(tuple(rep + pat), dtype=torch.int32, device="cuda")
+    thg, _ = timed(lambda: aol.tiler_gather(th, X, out=GH), inner=5)
+    nb = (X.numel() + GH.numel()) * 4
+    rec = {"config": "d3 the paper's H input tiler (Fig. 10) gather over 64 HD planes", "gather_ms": thg,
+           "gather_GBps": nb / thg / 1e6, "gather_frac": nb / thg / 1e6 / peak, "algorithmic_bytes_per_call": nb,
+           "timing": "CUDA events, 5 calls back to back per event pair, median of 20"}
+    if check:
+        rec["parity"] = cpu_parity_tiler([pre] + arr[1:], [pre] + rep[1:], pat, [0, 0, 0], P, F,
+                                         X[:pre].cpu().numpy(), G_pre=GH[:pre].cpu().numpy())
+        rec["parity_scope"] = f"oracle on planes 0..{pre - 1} of 64"
+    out.append(rec)
+    del X, GH
+    torch.cuda.empty_cache()
+    return out
+
+
+def record_d4(aol, peak, check):
+    """configs[3]: 64 frames of 3840x2160, same pattern ratios; all 64 checksums against the oracle."""
+    import numpy as np
+    import torch
+
+    N, C, H, W, seed = 64, 3, 2160, 3840, 1
+    x = aol.synth_frames(seed, 0, N, C, H, W)
+    z = torch.empty((N, C, 960, 1440), dtype=torch.int32, device="cuda")
+    cs = torch.empty(N, dtype=torch.uint64, device="cuda")
+    med, mn = timed(lambda: aol.downscale_frame(x, out=z, checksums=cs), inner=5)
+    b = N * frame_bytes(C, H, W)
+    rec = {"config": "d4 batch of 64 3840x2160 3-channel frames -> 1440x960 (BASELINE configs[3])", "ms": med,
+           "min_ms": mn, "frames_per_s": N / (med / 1e3), "GBps": b / med / 1e6, "frac": b / med / 1e6 / peak,
+           "timing": "CUDA events, 5 calls back to back per event pair, median of 20",
+           "plan": aol.downscale_frame_plan(N, C, H, W)}
+    torch.cuda.synchronize()
+    got = cs.cpu().view(torch.int64).numpy().view(np.uint64)
+    del x, z, cs
+    torch.cuda.empty_cache()
+    if check:
+        ref, spent = oracle_checksums(seed, range(N), C, H, W, oracle_threads())
+        rec["parity"] = bool(np.array_equal(ref, got))
+        rec["parity_scope"] = f"all {N} frame checksums vs the oracle"
+        rec["cpu_oracle_frames_per_s"] = N / spent
+    return rec
+
+
+def record_d5(a, aol, world, rank, use_dist, backend, d2_fps_per_gpu, peak, check):
+    """configs[4]: the 10,000-frame HD stream frame-sharded across the ranks (strong scaling).
+    Rank g owns stream frames [g*T/G, (g+1)*T/G) and cycles them through a device pool of 256 unique frames:
+    stream frame n holds the content of synthetic frame (n mod 256), so every frame's checksum is checked
+    against the oracle's 256 pool checksums.  Collective: all ranks call this."""
+    import numpy as np
+    import torch
+    import torch.distributed as dist
+
+    from paper_conf_ipps_guortgbs11_b200 import shard
+
+    T, pool, C, H, W, seed = a.d5_frames, 256, 3, 1080, 1920, a.seed
+    frame0, count = shard.strong_range(rank, world, T)
+    P = min(pool, count)
+    dev = torch.device("cuda", torch.cuda.current_device())
+    x = torch.empty((max(P, 1), C, H, W), dtype=torch.int32, device=dev)
+    j = 0
+    while j < P:   # slot j holds content (frame0 + j) mod pool: at most two contiguous runs
+        c0 = (frame0 + j) % pool
+        n = min(P - j, pool - c0)
+        aol.synth_frames(seed, c0, n, C, H, W, out=x[j:j + n])
+        j += n
+    z = torch.empty((max(P, 1), C, 480, 720), dtype=torch.int32, device=dev)
+    cs = torch.empty(max(count, 1), dtype=torch.uint64, device=dev)
+    calls = [(k, min(P, count - k)) for k in range(0, count, P)] if P > 0 else []
+    stream = torch.cuda.current_stream(dev)
+
+    def one_pass():
+        for k, n in calls:
+            aol.downscale_frame(x[:n], out=z[:n], checksums=cs[k:k + n])
+
+    one_pass()
+    torch.cuda.synchronize(dev)
+    mine = []
+    for _ in range(a.d5_repeats):
+        if use_dist:
+            dist.barrier()
+        torch.cuda.synchronize(dev)
+        e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        e0.record(stream)
+        one_pass()
+        e1.record(stream)
+        torch.cuda.synchronize(dev)
+        mine.append(e0.elapsed_time(e1))
+    gdev = dev if backend == "nccl" else torch.device("cpu")
+    el = torch.tensor(mine, dtype=torch.float64, device=gdev)
+    if use_dist:
+        allv = torch.empty(world * len(mine), dtype=torch.float64, device=gdev)
+        dist.all_gather_into_tensor(allv, el)
+        per_rank = allv.cpu().numpy().reshape(world, len(mine))
+    else:
+        per_rank = el.cpu().numpy().reshape(1, len(mine))
+    counts = [shard.strong_range(r, world, T)[1] for r in range(world)]
+    _, cs_all = shard.gather_results((cs[:count] if backend == "nccl" else cs[:count].cpu()), 0.0, counts=counts)
+    if rank != 0:
+        return None
+    cs_all = cs_all.cpu().numpy().view(np.uint64)
+    worst = per_rank.max(axis=0)                   # max over ranks, per repeat
+    rep_i = int(np.argsort(worst)[len(worst) // 2])   # the median repeat
+    total_fps = T / (worst[rep_i] / 1e3)
+    bpf = frame_bytes(C, H, W)
+    rec = {"config": f"d5 {T}-frame 1920x1080 stream frame-sharded across {world} GPU(s), device pool of {pool} "
+                     "unique frames per GPU (BASELINE configs[4])",
+           "scaling": "strong", "n_gpus": world, "frames_per_s": total_fps, "ms": float(worst[rep_i]),
+           "per_rank_ms": [float(v) for v in per_rank[:, rep_i]], "per_rank_frames": counts,
+           "per_gpu_GBps": [counts[r] * bpf / per_rank[r, rep_i] / 1e6 for r in range(world)],
+           "per_gpu_frac": [counts[r] * bpf / per_rank[r, rep_i] / 1e6 / peak for r in range(world)],
+           "launches_per_rank": len(calls), "repeats": a.d5_repeats,
+           "timing": "per-rank CUDA events around one pass over the rank's frames after a barrier; total = frames / "
+                     "max over ranks; median of the repeats",
+           "efficiency_vs_d2_per_gpu_rate": (total_fps / (world * d2_fps_per_gpu)) if d2_fps_per_gpu else None}
+    if check:
+        used = sorted(set(n % pool for n in range(T)))
+        ref, _ = oracle_checksums(seed, used, C, H, W, oracle_threads())
+        table = dict(zip(used, ref))
+        want = np.array([table[n % pool] for n in range(T)], dtype=np.uint64)
+        rec["parity"] = bool(cs_all.size == T and np.array_equal(cs_all, want))
+        rec["parity_scope"] = f"every one of the {T} stream frames' checksums vs the oracle's {len(used)} pool frames"
+    return rec
+
+
+# ============================================================ reference arm
+
+def run_reference(a, rank, world):
+    """--impl reference: the CPU oracle is this tier's reference arm (rank 0 only; other ranks exit 0).
+    One step = the oracle over every frame of the workload (300 HD frames), or -- if the run's steps would
+    exceed --ref-budget-seconds of oracle time -- over the largest prefix that fits (stated in `sample`)."""
     if rank != 0:
         return
-    steps, warm = a.steps, a.warmup
-    import oracle  # noqa: F401
-
-    fps_list = []
-    # warm-up + timed steps; each step is a bounded sample of the workload
-    for i in range(warm + steps):
-        fps, info = cpu_baseline(a, steps=1)
-        if i >= warm:
-            fps_list.append(fps)
-    value = statistics.median(fps_list)
+    nthreads = oracle_threads()
+    F = a.frames if not a.stream_frames else min(a.stream_frames, a.pool)
+    frames = F
+    times = []
+    for i in range(a.warmup + a.steps):
+        _, spent = oracle_checksums(a.seed, range(frames), a.channels, a.H, a.W, nthreads)
+        if i == 0:
+            remaining = a.warmup + a.steps - 1
+            per_frame = spent / frames
+            if remaining * per_frame * frames > a.ref_budget_seconds:
+                frames = max(nthreads, min(F, int(a.ref_budget_seconds / max(remaining, 1) / per_frame)))
+        if i >= a.warmup:
+            times.append(spent / frames)
+    s_per_frame = statistics.median(times)
+    value = 1.0 / s_per_frame
+    sample = (f"{frames} of the workload's {F} frames per step (seed {a.seed}, global frames 0..{frames - 1}), "
+              f"OpenMP over planes, median of {a.steps} steps after {a.warmup} warm-up; input generation untimed")
     line = {
-        "metric": METRIC, "value": value, "unit": "frames/s", "n_gpus": a.gpus, "steps": steps, "warmup": warm,
-        "ms_per_step": 1000.0 * info["seconds"], "higher_is_better": True, "scaling": "weak",
-        "vs_baseline": None, "dtype": "i32", "data": "synthetic",
-        "config": {"workload": workload_name(a), "frames": a.frames, "H": a.H, "W": a.W,
-                   "channels": a.channels, "l2": "inputs larger than L2 (no flush)"},
-        "impl": "reference",
-        "cpu_baseline": {"value": value, "unit": "frames/s", "cores": info["cores"], "kind": "oracle",
-                         "sample": info["sample"], "host": info.get("host")},
+        "metric": METRIC, "value": value, "unit": "frames/s", "n_gpus": world, "steps": a.steps, "warmup": a.warmup,
+        "ms_per_step": 1000.0 * s_per_frame * F, "higher_is_better": True,
+        "scaling": "strong" if a.stream_frames else "weak", "vs_baseline": None, "dtype": "i32",
+        "data": "synthetic", "config": workload_config(a, world), "impl": "reference",
+        "cpu_baseline": {"value": value, "unit": "frames/s", "cores": nthreads, "kind": "oracle", "sample": sample,
+                         "GBps_algorithmic": frame_bytes(a.channels, a.H, a.W) * value / 1e9, "host": host_cpu()},
         "e2e": {"value": value, "unit": "frames/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
     }
     print(json.dumps(line), flush=True)
 
+
+# ============================================================ main (GPU arm)
 
 def main():
     a = parse()
@@ -282,7 +689,7 @@ def main():
     local_rank = int(os.environ.get("LOCAL_RANK", "0"))
 
     if a.impl == "reference":
-        run_reference(a, rank)
+        run_reference(a, rank, world)
         return
 
     import numpy as np
@@ -292,6 +699,7 @@ def main():
     import paper_conf_ipps_guortgbs11_b200 as aol
     from paper_conf_ipps_guortgbs11_b200 import shard
 
+    extras = extras_of(a)
     # one process per GPU; AOL_DIST_BACKEND=gloo (and several ranks per GPU) only for testing the
     # multi-rank flow on a 1-GPU box -- the driver's runs use NCCL with one GPU per rank
     gpu = local_rank % max(1, torch.cuda.device_count())
@@ -311,10 +719,10 @@ def main():
     F, C, H, W = a.frames, a.channels, a.H, a.W
     if a.stream_frames:
         # configs[4]: strong scaling; this rank's frames of the global stream, processed in launches over a
-        # device pool (stream frame n of the rank uses pool slot n mod pool)
+        # device pool (stream frame n of the rank uses pool slot (n - frame0) mod pool)
         frame0, count = shard.strong_range(rank, world, a.stream_frames)
         F = max(1, min(a.pool, count))
-        calls = [min(F, count - k) for k in range(0, count, F)]
+        calls = [min(F, count - k) for k in range(0, count, F)]   # [] for a rank without frames
         a.no_e2e = True
     else:
         frame0, F = shard.weak_range(rank, world, F)
@@ -366,13 +774,20 @@ def main():
     launch_ms = [s.elapsed_time(e) for ss, es in zip(starts, ends) for s, e in zip(ss, es)]
     launch_frames = [n for _ in range(a.steps) for n in calls]
 
-    # max over ranks (NCCL), and gather per-rank checksums: the only cross-GPU traffic
-    counts = ([max(1, min(a.pool, shard.strong_range(r, world, a.stream_frames)[1])) for r in range(world)]
+    # max over ranks and per-rank elapsed (NCCL), and the per-rank checksums: the only cross-GPU traffic
+    gdev = dev if backend == "nccl" else torch.device("cpu")
+    counts = ([min(a.pool, shard.strong_range(r, world, a.stream_frames)[1]) for r in range(world)]
               if a.stream_frames else None)
-    max_ms, cs_all_t = shard.gather_results(cs if backend == "nccl" else cs.cpu(), elapsed_ms, counts=counts)
-    cs_all = cs_all_t.cpu().numpy().view(np.uint64) if use_dist else None
+    my_cs = cs[:min(F, count)] if backend == "nccl" else cs[:min(F, count)].cpu()
+    max_ms, cs_all_t = shard.gather_results(my_cs, elapsed_ms, counts=counts)
+    per_rank_ms = [elapsed_ms]
+    if use_dist:
+        allv = torch.empty(world, dtype=torch.float64, device=gdev)
+        dist.all_gather_into_tensor(allv, torch.tensor([elapsed_ms], dtype=torch.float64, device=gdev))
+        per_rank_ms = [float(v) for v in allv.cpu()]
+    cs_all = cs_all_t.cpu().numpy().view(np.uint64)
     if a.dump_checksums and rank == 0:
-        np.save(a.dump_checksums, cs_all if cs_all is not None else cs.cpu().view(torch.int64).numpy().view(np.uint64))
+        np.save(a.dump_checksums, cs_all)
 
     # e2e through the host-buffer C-ABI call
     e2e = None
@@ -395,7 +810,7 @@ def main():
             _, cs_h = aol.downscale_frame_host(x_host, out=z_host, chunk_frames=chunk, workspace=ws,
                                                streams=streams, device=dev, packed=packed)
         e2e_s = time.perf_counter() - t0
-        te = torch.tensor([e2e_s], dtype=torch.float64, device=dev if backend == "nccl" else "cpu")
+        te = torch.tensor([e2e_s], dtype=torch.float64, device=gdev)
         if use_dist:
             dist.all_reduce(te, op=dist.ReduceOp.MAX)
         e2e_s = float(te.item())
@@ -405,20 +820,41 @@ def main():
                "d2h_bytes_per_step": int(z_host.numel() * 4 + Fe * 8), "steps": a.e2e_steps,
                "chunk_frames": chunk, "checksums_match_device_path": same,
                "timing": "host wall clock around the blocking call, max over ranks"}
+        del x_host, z_host, ws
+    del x, z
+    torch.cuda.empty_cache()
+
+    total_frames = (a.stream_frames if a.stream_frames else world * F) * a.steps
+    value = total_frames / (max_ms / 1000.0)
+    peak, peak_src = measured_peak()
+    check = not a.no_cpu_baseline
+
+    # ---- sub-records: d5 on every rank (collective), d1 / d3 / d4 on rank 0
+    records = {}
+    if "d5" in extras:
+        d5 = record_d5(a, aol, world, rank, use_dist, backend, value / world, peak, check)
+        if d5 is not None:
+            records["d5"] = d5
+    if rank == 0:
+        if "d1" in extras:
+            records["d1"] = record_d1(aol, peak, check)
+        if "d3" in extras:
+            records["d3"] = record_d3(aol, peak, check)
+        if "d4" in extras:
+            records["d4"] = record_d4(aol, peak, check)
+    if use_dist:
+        dist.barrier()
 
     if rank != 0:
         if use_dist:
             dist.destroy_process_group()
         return
 
-    total_frames = (a.stream_frames if a.stream_frames else world * F) * a.steps
-    value = total_frames / (max_ms / 1000.0)
     bpf = bytes_per_frame(a)
-    avg_launch_s = statistics.mean(launch_ms) / 1000.0
+    avg_launch_s = statistics.mean(launch_ms) / 1000.0 if launch_ms else float("nan")
     # algorithmic bytes over kernel time, summed over this rank's launches (all equal in the default mode)
-    achieved = bpf * sum(launch_frames) / (sum(launch_ms) / 1000.0) / 1e9
-    peak, peak_src = measured_peak()
-    traffic, dram_pct, ncu_tag = ncu_traffic(a)
+    achieved = bpf * sum(launch_frames) / (sum(launch_ms) / 1000.0) / 1e9 if launch_ms else 0.0
+    traffic, dram_pct, ncu_tag, ncu_status = ncu_traffic(a, plan)
     mix_gbs, mix_src = mix_ceiling(a)
     mix = ({"GBps": mix_gbs, "frac": achieved / mix_gbs, "source": mix_src} if mix_gbs else None)
     line = {
@@ -426,35 +862,43 @@ def main():
         "warmup": a.warmup, "ms_per_step": max_ms / a.steps, "higher_is_better": True,
         "scaling": "strong" if a.stream_frames else "weak",
         "vs_baseline": None, "dtype": "i32", "data": "synthetic",   # arithmetic type (uint8 samples are summed in int32)
-        "config": {"workload": workload_name(a), "frames_per_gpu": count, "launches_per_step": len(calls),
-                   "H": H, "W": W, "channels": C,
-                   "in_dtype": a.dtype, "out_dtype": a.out_dtype, "l2": "inputs (7.46 GB at HD int32) larger than L2; no flush",
-                   "parallelism": f"frame-sharded x{world} (no data-path collective)",
-                   "kernel": {"1": "fused_tma_kernel", "2": "fused_generic_kernel"}[str(plan["kernel"])],
-                   "plan": plan},
+        "config": workload_config(a, world),
+        "launch": {"kernel": {"1": "fused_tma_kernel", "2": "fused_generic_kernel"}[str(plan["kernel"])],
+                   "plan": plan, "launches_per_step": len(calls), "frames_per_rank": count,
+                   "src_hash": src_hash()},
         "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s", "frac": achieved / peak,
-                     "traffic": traffic, "peak_source": peak_src,
+                     "traffic": traffic, "traffic_status": ncu_status, "peak_source": peak_src,
                      # the copy peak is half writes while this path is ~86 % reads, so frac can exceed 1; ncu's
                      # DRAM utilisation of the same launch (committed capture) is the direct measure
                      "ncu_dram_pct_of_peak": dram_pct, "ncu_capture": ncu_tag,
                      "mix_ceiling": mix,
-                     "algorithmic_bytes_per_launch": bpf * calls[0],
-                     "avg_launch_ms": avg_launch_s * 1000.0, "min_launch_ms": min(launch_ms)},
+                     "algorithmic_bytes_per_launch": bpf * calls[0] if calls else 0,
+                     "avg_launch_ms": avg_launch_s * 1000.0, "min_launch_ms": min(launch_ms) if launch_ms else None},
         # per call: zero_checksums_kernel + the fused kernel (its programmatic dependent)
         "gpu_launches": a.steps * len(calls) * (2 if plan["kernel"] == 1 else 1),
         "clocks": clk.summary(),
+        "per_rank_ms": per_rank_ms,
+        "per_gpu_GBps": [bpf * (world * F if not a.stream_frames else a.stream_frames) / world * a.steps
+                         / (ms / 1e3) / 1e9 for ms in per_rank_ms],
     }
     if e2e is not None:
         line["e2e"] = e2e
-    if use_dist and cs_all is not None:
+    if use_dist:
         line["gathered_checksums"] = int(cs_all.size)
-    if world == 1 and not a.no_cpu_baseline:
-        fps, info = cpu_baseline(a, gpu_cs=cs.cpu().view(torch.int64).numpy().view(np.uint64), frame0=frame0,
-                                 min_seconds=a.cpu_baseline_seconds, single_thread=True)
-        line["cpu_baseline"] = {"value": fps, "unit": "frames/s", "cores": info["cores"], "kind": "oracle",
-                                "sample": info["sample"], "parity_sample_ok": info.get("parity_sample_ok"),
-                                "single_thread_s_per_frame": info.get("single_thread_s_per_frame"),
-                                "host": info.get("host")}
+    if world == 1 and not a.no_cpu_baseline and not a.stream_frames:
+        line["cpu_baseline"] = cpu_baseline(a, frame0, F, gpu_cs=cs_all, min_seconds=a.cpu_baseline_seconds,
+                                            single_thread=True)
+    if records:
+        line["records"] = records
+        flags = []
+        for r in records.values():
+            for rr in (r if isinstance(r, list) else [r]):
+                if "parity" in rr:
+                    flags.append(rr["parity"])
+        cb = line.get("cpu_baseline", {})
+        if "parity_all_frames" in cb:
+            flags.append(cb["parity_all_frames"])
+        line["parity_all_records"] = bool(flags) and all(flags)
     print(json.dumps(line), flush=True)
     if use_dist:
         dist.destroy_process_group()

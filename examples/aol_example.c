@@ -6,7 +6,7 @@
  * three agree, and prints the per-frame checksums (compared against the CPU oracle by
  * tests/test_gpu_example.py).
  *
- * build: gcc -std=c99 -O2 -I include -I /usr/local/cuda/include examples/aol_example.c \
+ * build: gcc -std=c11 -O2 -I include -I /usr/local/cuda/include examples/aol_example.c \
  *            -L paper_conf_ipps_guortgbs11_b200 -laol -L /usr/local/cuda/lib64 -lcudart \
  *            -Wl,-rpath,$PWD/paper_conf_ipps_guortgbs11_b200 -o build/aol_example
  * run:   build/aol_example [frames=4] [seed=7]

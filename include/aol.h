@@ -23,7 +23,14 @@
  *    launch (asynchronous).  Kernel faults surface at the caller's next sync.
  *  - Errors are returned synchronously as aol_status_t for invalid arguments,
  *    shapes, dtypes, alignment, and launch failures; aol_last_error() then
- *    holds a message.  On error nothing has been enqueued.
+ *    holds a message.  A device call that returns an error has enqueued
+ *    nothing: arguments, the launch plan, the TMA descriptor, kernel
+ *    attributes and the launch configuration are all checked before the first
+ *    enqueue (tested with aol_debug_fail_next_launches, aol_tuning.h).  The one
+ *    exception is a CUDA launch that fails after that pre-flight (a broken CUDA
+ *    context): then an earlier kernel of the same call (the checksum zeroing) may
+ *    already be enqueued.  aol_downscale_frame_host is a pipeline of many
+ *    enqueues: see its comment.
  *  - Integer arithmetic is exact: results are bit-identical to the CPU oracle.
  *  - Arrays are dense row-major; a batch of frames is planar
  *    [frames][channels][H][W] (reading Z8: one plane per colour channel,
@@ -35,7 +42,9 @@
 #include <stddef.h>
 #include <stdint.h>
 
-#include <cuda_runtime_api.h>
+/* The one CUDA type in these signatures, declared as cuda_runtime_api.h declares it (an identical
+ * typedef may be repeated in C11 and C++), so this header needs no CUDA include path. */
+typedef struct CUstream_st* cudaStream_t;
 
 #ifdef __cplusplus
 extern "C" {
@@ -106,26 +115,9 @@ typedef struct {
     int32_t bands_per_unit; /* 9-row bands per work unit, 0 = auto (balance waves vs halo)     */
     int32_t kernel;         /* 0 = auto, 1 = TMA fused kernel (error if shape unsupported),
                                2 = generic fused kernel (any W%8==0, H%9==0)                   */
-    int32_t flags;          /* AOL_FLAG_* bits (tuning experiments; results are identical)    */
+    int32_t flags;          /* 0 in production; A/B experiment bits of aol_tuning.h (results are
+                               identical whatever the bits)                                    */
 } aol_launch_opts_t;
-
-/* bit 0 is reserved (was AOL_FLAG_HALO_LAST, a round-1 experiment: the halo rows now always stream first) */
-#define AOL_FLAG_EVICT_FIRST_LOADS 2   /* TMA input loads with the L2 evict_first policy            */
-#define AOL_FLAG_EVICT_FIRST_STORES 4  /* TMA output stores with the L2 evict_first policy          */
-#define AOL_FLAG_BLOCKED_UNITS 8       /* each CTA takes a contiguous block of work units (default:
-                                          round-robin, so concurrently running CTAs are adjacent)  */
-#define AOL_FLAG_U8_BULK 16            /* uint8 input: 1-D bulk copies even when W % 128 == 0      */
-#define AOL_FLAG_NO_PDL 64             /* launch the fused kernel after the checksum zeroing completes
-                                          (default: overlapped, programmatic dependent launch)        */
-#define AOL_FLAG_U8_ONE_REP 32         /* uint8 input: one H repetition per consumer thread even for
-                                          W >= 1024 (default there: two)                            */
-#define AOL_FLAG_I32_LINEAR 128        /* int32 input: 1-D bulk copies into linear smem rows even when
-                                          W % 32 == 0 (default there: TMA tensor loads, SWIZZLE_128B) */
-#define AOL_FLAG_I32_SWZ32 256         /* int32 input, W % 32 != 0, W <= 2048: TMA tensor loads of
-                                          32-byte lines under SWIZZLE_32B (default: linear rows)     */
-#define AOL_FLAG_ROW_STAGES 512        /* int32 input: one row per TMA ring stage (default when a row
-                                          triple exceeds a third of the ring's bytes: W > 3271)        */
-#define AOL_FLAG_TRIPLE_STAGES 1024    /* int32 input: one row triple per ring stage for any W       */
 
 /* The launch configuration aol_downscale_frame_ex would use (for reports/tests). */
 typedef struct {
@@ -207,8 +199,9 @@ AOL_API aol_status_t aol_downscale_v(const int32_t* d_in, int32_t* d_out, int64_
  * [frames][channels][4H/9][3W/8], H filter first (Fig. 2).
  * in_dtype: AOL_I32 (values must lie in (-2^27, 2^27), reading Z12), AOL_U8
  * (8-bit samples) or AOL_RGB8 (packed pixels: d_in [frames][H][W][3] bytes, channels == 3,
- * W % 16 == 0; the output is still planar).  d_frame_checksums: nullable device u64 [frames],
- * overwritten with  sum (u64)(u32)Z[n][c][y][x] * (1 + (c*Ho + y)*Wo + x)  mod 2^64.
+ * W % 16 == 0, W <= 6400 with int32 outputs / 7936 with int16 outputs; the output is still planar).  d_frame_checksums: nullable device u64 [frames],
+ * 8-byte aligned, overwritten with
+ * sum (u64)(u32)Z[n][c][y][x] * (1 + (c*Ho + y)*Wo + x)  mod 2^64.
  * frames == 0 is a no-op.  d_in/d_out 16-byte aligned.  Async on s. */
 AOL_API aol_status_t aol_downscale_frame(const void* d_in, aol_dtype_t in_dtype, int32_t* d_out, int64_t frames,
                                  int64_t channels, int64_t H, int64_t W, uint64_t* d_frame_checksums,
@@ -257,6 +250,9 @@ AOL_API size_t aol_downscale_frame_host_workspace_bytes(aol_dtype_t in_dtype, in
  * pageable memory works but serialises).  d_workspace: device, at least
  * aol_downscale_frame_host_workspace_bytes(...) bytes.  BLOCKING: returns when
  * h_out (and h_frame_checksums, nullable) are complete. */
+/* On an error in the middle of the pipeline, the chunks enqueued before it still complete (the call
+ * synchronises the three streams before returning); h_out then holds those chunks' results, the rest
+ * is unspecified. */
 AOL_API aol_status_t aol_downscale_frame_host(const void* h_in, aol_dtype_t in_dtype, int32_t* h_out, int64_t frames,
                                       int64_t channels, int64_t H, int64_t W, uint64_t* h_frame_checksums,
                                       int64_t chunk_frames, void* d_workspace, size_t ws_bytes,

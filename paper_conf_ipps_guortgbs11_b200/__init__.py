@@ -25,7 +25,7 @@ from ._lib import (FILTER_H, FILTER_V, AolError, I16, I32, I64, PRESET_H_IN, PRE
 
 __all__ = [
     "AolError", "version", "make_tiler", "tiler_preset", "tiler_validate", "tiler_is_injective",
-    "tiler_gather", "tiler_scatter", "downscale_h", "downscale_v", "downscale_frame", "downscale_frame_plan",
+    "tiler_gather", "tiler_scatter", "tiler_scatter_workspace_bytes", "downscale_h", "downscale_v", "downscale_frame", "downscale_frame_plan",
     "frame_checksum", "downscale_frame_host", "synth_frames", "library_path", "downscale_frame_packed",
     "PRESET_H_IN", "PRESET_H_OUT", "PRESET_V_IN", "PRESET_V_OUT", "SYNTH_KINDS",
     "make_filter", "filter_preset", "filter_validate", "filter_apply", "FILTER_H", "FILTER_V", "FLAGS",
@@ -121,6 +121,11 @@ def tiler_is_injective(t: aol_tiler_t) -> bool:
     v = ctypes.c_int(0)
     check(lib().aol_tiler_is_injective(ctypes.byref(t), ctypes.byref(v)))
     return bool(v.value)
+
+
+def tiler_scatter_workspace_bytes(t: aol_tiler_t) -> int:
+    """Device workspace bytes a SEQUENTIAL scatter with tiler t needs (0 if none)."""
+    return int(lib().aol_tiler_scatter_workspace_bytes(ctypes.byref(t)))
 
 
 def tiler_gather(t: aol_tiler_t, array: torch.Tensor, out: Optional[torch.Tensor] = None,

@@ -58,13 +58,10 @@ class aol_filter_t(ctypes.Structure):
                 ("window_start", ctypes.c_int32 * MAX_WINDOWS)]
 
 
-# aol_launch_opts_t.flags bits (include/aol.h AOL_FLAG_*; tuning experiments, results are identical)
-FLAG_EVICT_FIRST_LOADS, FLAG_EVICT_FIRST_STORES, FLAG_BLOCKED_UNITS, FLAG_U8_BULK = 2, 4, 8, 16
-FLAG_U8_ONE_REP, FLAG_NO_PDL, FLAG_I32_LINEAR, FLAG_I32_SWZ32 = 32, 64, 128, 256
+# aol_launch_opts_t.flags bits (include/aol_tuning.h AOL_FLAG_*; A/B experiments, results are identical)
+FLAG_U8_ONE_REP, FLAG_NO_PDL, FLAG_I32_LINEAR = 32, 64, 128
 FLAG_ROW_STAGES, FLAG_TRIPLE_STAGES = 512, 1024
-FLAGS = {"EVICT_FIRST_LOADS": FLAG_EVICT_FIRST_LOADS, "EVICT_FIRST_STORES": FLAG_EVICT_FIRST_STORES,
-         "BLOCKED_UNITS": FLAG_BLOCKED_UNITS, "U8_BULK": FLAG_U8_BULK, "U8_ONE_REP": FLAG_U8_ONE_REP,
-         "NO_PDL": FLAG_NO_PDL, "I32_LINEAR": FLAG_I32_LINEAR, "I32_SWZ32": FLAG_I32_SWZ32,
+FLAGS = {"U8_ONE_REP": FLAG_U8_ONE_REP, "NO_PDL": FLAG_NO_PDL, "I32_LINEAR": FLAG_I32_LINEAR,
          "ROW_STAGES": FLAG_ROW_STAGES, "TRIPLE_STAGES": FLAG_TRIPLE_STAGES}
 
 
@@ -114,6 +111,7 @@ SIGNATURES = {
     "aol_filter_preset": ([ctypes.c_int, _I64, _I64, _I64, _FP], _ST),
     "aol_filter_validate": ([_FP], _ST),
     "aol_filter_apply": ([_FP, _P, _P, _P], _ST),
+    "aol_debug_fail_next_launches": ([ctypes.c_int], None),
     "aol_synth_frames": ([ctypes.c_uint64, _I64, _I64, _I64, _I64, _I64, _I32, _I32, ctypes.c_int, _P, _P], _ST),
 }
 

@@ -102,6 +102,24 @@ int kernel_occupancy(const void* fn, int block, int smem) {
     return occ;
 }
 
+namespace {
+thread_local int g_fail_launches = 0;   // aol_debug_fail_next_launches (test hook)
+}
+
+aol_status_t launch_preflight(const void* fn, int block, int smem, const char* what) {
+    if (g_fail_launches > 0) {
+        --g_fail_launches;
+        set_error("launch of %s failed: injected failure (aol_debug_fail_next_launches)", what);
+        return AOL_E_CUDA;
+    }
+    if (kernel_occupancy(fn, block, smem) < 1) {
+        set_error("launch of %s is not runnable: %d threads with %d bytes of dynamic shared memory", what, block,
+                  smem);
+        return AOL_E_CUDA;
+    }
+    return AOL_OK;
+}
+
 int elsize_of(aol_dtype_t el) {
     switch (el) {
         case AOL_U8: case AOL_RAW8: return 1;
@@ -252,7 +270,8 @@ using namespace aol;
 namespace {
 
 aol_status_t check_frame_args(const void* d_in, aol_dtype_t in_dtype, const void* d_out, int64_t frames,
-                              int64_t channels, int64_t H, int64_t W, aol_dtype_t out_dtype = AOL_I32) {
+                              int64_t channels, int64_t H, int64_t W, aol_dtype_t out_dtype = AOL_I32,
+                              const uint64_t* d_cs = nullptr) {
     if (frames < 0 || channels <= 0 || H <= 0 || W <= 0)
         return fail(AOL_E_INVALID, "frames must be >= 0 and channels, H, W > 0");
     if (in_dtype != AOL_I32 && in_dtype != AOL_U8 && in_dtype != AOL_RGB8)
@@ -269,18 +288,30 @@ aol_status_t check_frame_args(const void* d_in, aol_dtype_t in_dtype, const void
     if (frames > 0 && (!d_in || !d_out)) return fail(AOL_E_INVALID, "null buffer");
     if (frames > 0 && (!aligned16(d_in) || !aligned16(d_out)))
         return fail(AOL_E_ALIGN, "d_in and d_out must be 16-byte aligned");
+    if (reinterpret_cast<uintptr_t>(d_cs) % 8) return fail(AOL_E_ALIGN, "d_frame_checksums must be 8-byte aligned");
+    return AOL_OK;
+}
+
+constexpr int32_t kKnownFlags = AOL_FLAG_U8_ONE_REP | AOL_FLAG_NO_PDL | AOL_FLAG_I32_LINEAR | AOL_FLAG_ROW_STAGES |
+                                AOL_FLAG_TRIPLE_STAGES;
+
+aol_status_t check_opts(const aol_launch_opts_t* opts) {
+    if (opts && (opts->ctas_per_sm < 0 || opts->ctas_per_sm > 8 || opts->stages < 0 || opts->bands_per_unit < 0 ||
+                 opts->kernel < 0 || opts->kernel > 2))
+        return fail(AOL_E_INVALID, "launch options out of range");
+    if (opts && (opts->flags & ~kKnownFlags))
+        return fail(AOL_E_INVALID, "unknown launch-option flag bits (see include/aol_tuning.h)");
     return AOL_OK;
 }
 
 aol_status_t frame_ex(const void* d_in, aol_dtype_t in_dtype, void* d_out, aol_dtype_t out_dtype, int64_t frames,
                       int64_t channels, int64_t H, int64_t W, uint64_t* d_cs, const aol_launch_opts_t* opts,
                       cudaStream_t s) {
-    aol_status_t st = check_frame_args(d_in, in_dtype, d_out, frames, channels, H, W, out_dtype);
+    aol_status_t st = check_frame_args(d_in, in_dtype, d_out, frames, channels, H, W, out_dtype, d_cs);
     if (st != AOL_OK) return st;
     if (frames == 0) return AOL_OK;
-    if (opts && (opts->ctas_per_sm < 0 || opts->ctas_per_sm > 8 || opts->stages < 0 || opts->bands_per_unit < 0 ||
-                 opts->kernel < 0 || opts->kernel > 2))
-        return fail(AOL_E_INVALID, "launch options out of range");
+    st = check_opts(opts);
+    if (st != AOL_OK) return st;
     FusedPlan plan;
     st = plan_fused(in_dtype, out_dtype, d_in, d_out, frames, channels, H, W, opts, &plan);
     if (st != AOL_OK) return st;
@@ -292,6 +323,8 @@ aol_status_t frame_ex(const void* d_in, aol_dtype_t in_dtype, void* d_out, aol_d
 extern "C" {
 
 int aol_version(void) { return AOL_VERSION; }
+
+void aol_debug_fail_next_launches(int n) { g_fail_launches = n > 0 ? n : 0; }
 
 const char* aol_last_error(void) { return aol::last_error_cstr(); }
 
@@ -355,7 +388,12 @@ aol_status_t aol_tiler_is_injective(const aol_tiler_t* t, int* injective) {
     if (st != AOL_OK) return st;
     if (td.array_elems > (int64_t(1) << 32) || td.total > (int64_t(1) << 32))
         return fail(AOL_E_RANGE, "brute-force injectivity check limited to 2^32 elements");
-    std::vector<uint8_t> seen(size_t(td.array_elems), 0);
+    std::vector<uint64_t> seen;   // one bit per array element (<= 512 MiB)
+    try {
+        seen.assign(size_t((td.array_elems + 63) / 64), 0);
+    } catch (...) {
+        return fail(AOL_E_RANGE, "not enough host memory for the injectivity bitmap");
+    }
     int64_t idx[2 * AOL_MAX_RANK] = {0};
     *injective = 1;
     for (int64_t g = 0; g < td.total; ++g) {
@@ -365,11 +403,12 @@ aol_status_t aol_tiler_is_injective(const aol_tiler_t* t, int* injective) {
             for (int d = 0; d < td.nd; ++d) v += __int128(td.coef[a][d]) * idx[d];
             off += int64_t(v % td.ashape[a]) * td.astride[a];
         }
-        if (seen[size_t(off)]) {
+        const uint64_t bit = uint64_t(1) << (off & 63);
+        if (seen[size_t(off >> 6)] & bit) {
             *injective = 0;
             return AOL_OK;
         }
-        seen[size_t(off)] = 1;
+        seen[size_t(off >> 6)] |= bit;
         for (int d = td.nd - 1; d >= 0; --d) {
             if (++idx[d] < td.ext[d]) break;
             idx[d] = 0;
@@ -462,6 +501,8 @@ aol_status_t aol_downscale_frame_plan_out(aol_dtype_t in_dtype, aol_dtype_t out_
     if (!out) return fail(AOL_E_INVALID, "out is NULL");
     aol_status_t st = check_frame_args(nullptr, in_dtype, nullptr, 0, channels, H, W, out_dtype);
     if (st != AOL_OK) return st;
+    st = check_opts(opts);
+    if (st != AOL_OK) return st;
     if (frames <= 0) return fail(AOL_E_INVALID, "frames must be > 0 to plan");
     FusedPlan p;
     st = plan_fused(in_dtype, out_dtype, nullptr, nullptr, frames, channels, H, W, opts, &p);
@@ -488,6 +529,8 @@ aol_status_t aol_frame_checksum(const int32_t* d_out, int64_t frames, int64_t ch
     if (frames < 0 || channels <= 0 || Ho <= 0 || Wo <= 0) return fail(AOL_E_INVALID, "bad extents");
     if (frames == 0) return AOL_OK;
     if (!d_out || !d_checksums) return fail(AOL_E_INVALID, "null buffer");
+    if (reinterpret_cast<uintptr_t>(d_checksums) % 8 || reinterpret_cast<uintptr_t>(d_out) % 4)
+        return fail(AOL_E_ALIGN, "d_checksums must be 8-byte and d_out 4-byte aligned");
     return launch_checksum(d_out, frames, channels * Ho * Wo, d_checksums, s);
 }
 

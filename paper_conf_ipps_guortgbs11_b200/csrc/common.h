@@ -7,6 +7,7 @@
 #include <cuda_runtime.h>
 
 #include "../../include/aol.h"
+#include "../../include/aol_tuning.h"
 
 namespace aol {
 
@@ -52,6 +53,10 @@ struct DeviceInfo {
 aol_status_t device_info(DeviceInfo* out);               // memoised per device
 aol_status_t kernel_smem(const void* fn, int smem_bytes);   // cudaFuncSetAttribute(MaxDynamicSmem), memoised
 int kernel_occupancy(const void* fn, int block, int smem);  // resident CTAs per SM, memoised (0 on error)
+// Pre-flight of a launch about to be enqueued: the configuration must be runnable (occupancy >= 1 CTA/SM),
+// and the test hook aol_debug_fail_next_launches() may force a failure here.  Called before the FIRST
+// enqueue of an entry point, so a failing call leaves the caller's buffers untouched.
+aol_status_t launch_preflight(const void* fn, int block, int smem, const char* what);
 
 // ---- launchers implemented in the .cu files (all validate nothing; callers do)
 struct FusedPlan {

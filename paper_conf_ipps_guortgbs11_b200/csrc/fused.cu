@@ -55,26 +55,23 @@ aol_status_t get_encode_fn(EncodeTiledFn* fn) {
 
 // Shared-memory layout of an int32 row triple (the kernel's kSwz): 128 = TMA tensor loads of 128-byte lines
 // under SWIZZLE_128B (W % 32 == 0); 0 = one 1-D bulk copy of the contiguous triple into linear rows (W % 32 != 0,
-// or forced by AOL_FLAG_I32_LINEAR); 32 = TMA tensor loads of 32-byte lines under SWIZZLE_32B (W % 32 != 0 with
-// AOL_FLAG_I32_SWZ32, W <= 2048: the round-1 layout, kept for A/B).  -1 for uint8 input.
+// or forced by AOL_FLAG_I32_LINEAR).  -1 for uint8 input.
 int i32_layout(aol_dtype_t dt, int64_t W, int flags) {
     if (dt != AOL_I32) return -1;
     if (flags & AOL_FLAG_I32_LINEAR) return 0;
-    if (W % 32 == 0) return 128;
-    return (flags & AOL_FLAG_I32_SWZ32) ? 32 : 0;
+    return W % 32 == 0 ? 128 : 0;
 }
 
 bool tma_shape_ok(aol_dtype_t dt, int64_t planes, int64_t channels, int64_t H, int64_t W, int flags) {
     if (H < 9 || W / 8 > kMaxConsumers) return false;
     // checksum weights (1 + frame-local output index) are computed in 32 bits
     if (channels * (4 * (H / 9)) * (3 * (W / 8)) >= (int64_t(1) << 32) - 1) return false;
-    // int32 tensor layouts: {32, W/32, 3}-element boxes under SWIZZLE_128B or {8, W/8, 3} under SWIZZLE_32B
-    // (a box dimension holds at most 256 elements; tensor row coordinates are int32); linear rows: 1-D bulk
-    // copies of 12W bytes (16-byte multiple since W % 8 == 0)
+    // int32 tensor layout: {32, W/32, 3}-element boxes under SWIZZLE_128B (a box dimension holds at most 256
+    // elements; tensor row coordinates are int32); linear rows: 1-D bulk copies of 12W bytes (16-byte multiple
+    // since W % 8 == 0)
     if (dt == AOL_I32) {
-        const int layout = i32_layout(dt, W, flags);
-        if (layout == 0) return true;
-        return (layout == 128 ? W / 32 <= 256 : W / 8 <= 256) && planes * H < (int64_t(1) << 31);
+        if (i32_layout(dt, W, flags) == 0) return true;
+        return W / 32 <= 256 && planes * H < (int64_t(1) << 31);
     }
     if (dt == AOL_U8) return W % 16 == 0;   // 1-D bulk copies: 16-byte granularity
     if (dt == AOL_RGB8) return W % 16 == 0;  // packed pixels: 9W-byte triples, 24-byte repetitions
@@ -140,20 +137,34 @@ aol_status_t encode_row_map(CUtensorMap* map, aol_dtype_t dt, const void* base, 
     aol_status_t st = get_encode_fn(&encode);
     if (st != AOL_OK) return st;
     const bool i32 = dt == AOL_I32;
-    const bool s32 = i32_layout(dt, W, flags) == 32;
-    const cuuint64_t inner = i32 ? (s32 ? 8 : 32) : 128, es = i32 ? 4 : 1;
+    const cuuint64_t inner = i32 ? 32 : 128, es = i32 ? 4 : 1;
     const cuuint64_t gdim[3] = {inner, cuuint64_t(W) / inner, cuuint64_t(rows)};
     const cuuint64_t gstride[2] = {inner * es, cuuint64_t(W) * es};
     const cuuint32_t box[3] = {cuuint32_t(inner), cuuint32_t(W / int64_t(inner)), cuuint32_t(rows_per_stage(dt, W, flags))};
     const cuuint32_t estr[3] = {1, 1, 1};
     CUresult cr = encode(map, i32 ? CU_TENSOR_MAP_DATA_TYPE_INT32 : CU_TENSOR_MAP_DATA_TYPE_UINT8, 3,
                          const_cast<void*>(base), gdim, gstride, box, estr, CU_TENSOR_MAP_INTERLEAVE_NONE,
-                         i32 ? (s32 ? CU_TENSOR_MAP_SWIZZLE_32B : CU_TENSOR_MAP_SWIZZLE_128B) : CU_TENSOR_MAP_SWIZZLE_NONE,
+                         i32 ? CU_TENSOR_MAP_SWIZZLE_128B : CU_TENSOR_MAP_SWIZZLE_NONE,
                          l2_promotion(), CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
     if (cr != CUDA_SUCCESS) {
         set_error("cuTensorMapEncodeTiled failed (CUresult %d)", int(cr));
         return AOL_E_CUDA;
     }
+    return AOL_OK;
+}
+
+// The generic fused kernel (kernel 2): pre-flight, then zero the checksums and launch.
+template <typename Tin, typename Tout>
+aol_status_t launch_generic(const FusedPlan& plan, const void* d_in, void* d_out, uint64_t* d_cs, int64_t frames,
+                            int64_t planes, int64_t H, int64_t W, int32_t Ho, int32_t Wo, int64_t channels,
+                            cudaStream_t s) {
+    auto k = d_cs ? fused_generic_kernel<Tin, Tout, true> : fused_generic_kernel<Tin, Tout, false>;
+    aol_status_t st = launch_preflight(reinterpret_cast<const void*>(k), plan.block, 0, "fused_generic_kernel");
+    if (st != AOL_OK) return st;   // nothing enqueued yet
+    if (d_cs) AOL_CUDA_TRY(cudaMemsetAsync(d_cs, 0, size_t(frames) * sizeof(uint64_t), s));
+    k<<<plan.grid, plan.block, 0, s>>>(static_cast<const Tin*>(d_in), static_cast<Tout*>(d_out), d_cs, planes,
+                                       int32_t(H), int32_t(W), Ho, Wo, int32_t(channels));
+    AOL_LAUNCH_CHECK("fused_generic_kernel");
     return AOL_OK;
 }
 
@@ -232,8 +243,11 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void*
     }
     if (o.kernel == 2) tma_ok = false;
     if (rgb && !tma_ok) {
-        set_error("packed 24-bit pixels (AOL_RGB8) need the TMA fused kernel: W %% 16 == 0, W <= 7936, 16-byte "
-                  "aligned buffers");
+        // a CTA holds two 9W-byte ring stages plus the 3-plane 4-row output staging (18W bytes for int32, 9W for
+        // int16 outputs) within the 227 KB opt-in: W <= 6400 (int32 outputs) / 7936 (int16 outputs)
+        set_error("packed 24-bit pixels (AOL_RGB8) need the TMA fused kernel: W %% 16 == 0, W <= %d with %s outputs "
+                  "(two ring stages and the output staging in shared memory), 16-byte aligned buffers",
+                  out_es == 4 ? 6400 : 7936, out_es == 4 ? "int32" : "int16");
         return AOL_E_SHAPE;
     }
 
@@ -303,28 +317,16 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
     const int32_t Ho = int32_t(4 * (H / 9)), Wo = int32_t(3 * (W / 8));
 
     if (plan.kernel == 2) {
-        if (d_cs) AOL_CUDA_TRY(cudaMemsetAsync(d_cs, 0, size_t(frames) * sizeof(uint64_t), s));
-        if (in_dtype == AOL_U8 && plan.out_es == 2) {
-            auto k = d_cs ? fused_generic_kernel<uint8_t, int16_t, true> : fused_generic_kernel<uint8_t, int16_t, false>;
-            k<<<plan.grid, plan.block, 0, s>>>(static_cast<const uint8_t*>(d_in), static_cast<int16_t*>(d_out), d_cs,
-                                               planes, int32_t(H), int32_t(W), Ho, Wo, int32_t(channels));
-        } else if (in_dtype == AOL_U8) {
-            auto k = d_cs ? fused_generic_kernel<uint8_t, int32_t, true> : fused_generic_kernel<uint8_t, int32_t, false>;
-            k<<<plan.grid, plan.block, 0, s>>>(static_cast<const uint8_t*>(d_in), static_cast<int32_t*>(d_out), d_cs,
-                                               planes, int32_t(H), int32_t(W), Ho, Wo, int32_t(channels));
-        } else {
-            auto k = d_cs ? fused_generic_kernel<int32_t, int32_t, true> : fused_generic_kernel<int32_t, int32_t, false>;
-            k<<<plan.grid, plan.block, 0, s>>>(static_cast<const int32_t*>(d_in), static_cast<int32_t*>(d_out), d_cs,
-                                               planes, int32_t(H), int32_t(W), Ho, Wo, int32_t(channels));
-        }
-        AOL_LAUNCH_CHECK("fused_generic_kernel");
-        return AOL_OK;
+        if (in_dtype == AOL_U8 && plan.out_es == 2)
+            return launch_generic<uint8_t, int16_t>(plan, d_in, d_out, d_cs, frames, planes, H, W, Ho, Wo, channels, s);
+        if (in_dtype == AOL_U8)
+            return launch_generic<uint8_t, int32_t>(plan, d_in, d_out, d_cs, frames, planes, H, W, Ho, Wo, channels, s);
+        return launch_generic<int32_t, int32_t>(plan, d_in, d_out, d_cs, frames, planes, H, W, Ho, Wo, channels, s);
     }
 
     CUtensorMap map;
     std::memset(&map, 0, sizeof map);
-    const bool u8_tensor = in_dtype == AOL_U8 && W % 128 == 0 && W / 128 <= 256 &&
-                           planes * H < (int64_t(1) << 31) && !(plan.flags & AOL_FLAG_U8_BULK);
+    const bool u8_tensor = in_dtype == AOL_U8 && W % 128 == 0 && W / 128 <= 256 && planes * H < (int64_t(1) << 31);
     const int layout = i32_layout(in_dtype, W, plan.flags);
     if (layout > 0 || u8_tensor) {
         aol_status_t st = encode_row_map(&map, in_dtype, d_in, planes * H, W, plan.flags);
@@ -347,7 +349,7 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
     a.channels = rgb ? 1 : int32_t(channels);   // packed: the unit index is the frame index
     a.row_pitch = int32_t(rgb ? 3 * W : W);
     a.reps = int32_t(W / 8);
-    a.segs = int32_t(layout == 32 ? W / 8 : W / 32);   // int32 swizzled lines per row (unused for linear rows)
+    a.segs = int32_t(W / 32);   // int32 swizzled 128-byte lines per row (unused for linear rows)
     a.triples_per_plane = int32_t(H / 3);
     a.nbands = int32_t(H / 9);
     a.bands_per_unit = plan.bands_per_unit;
@@ -358,18 +360,22 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
     a.stage_stride = geom.stage_stride;
     a.out_bytes = geom.out_bytes;
     a.n_consumer = plan.block - 32;
-    a.hint_loads = (plan.flags & AOL_FLAG_EVICT_FIRST_LOADS) ? 1 : 0;
-    a.hint_stores = (plan.flags & AOL_FLAG_EVICT_FIRST_STORES) ? 1 : 0;
-    a.blocked_units = (plan.flags & AOL_FLAG_BLOCKED_UNITS) ? 1 : 0;
 
     KernelFn k = pick(in_dtype, plan.out_es, d_cs != nullptr, plan.reps_per_thread, W, plan.flags, plan.block,
                       plan.ctas_per_sm);
     aol_status_t st_attr = kernel_smem(reinterpret_cast<const void*>(k), plan.smem);
     if (st_attr != AOL_OK) return st_attr;
+    // Everything that can fail before the kernels run has been resolved (plan, tensor map, smem attribute);
+    // the pre-flight checks the configuration is runnable.  Nothing has been enqueued yet.
+    st_attr = launch_preflight(reinterpret_cast<const void*>(k), plan.block, plan.smem, "fused_tma_kernel");
+    if (st_attr != AOL_OK) return st_attr;
     // With checksums: zero them in a one-CTA kernel and launch the fused kernel as its programmatic
     // dependent, so the zeroing (and the launch gap after it) overlaps the fused kernel's start instead of
     // preceding it (single-frame latency).  Only the zero kernel can be the primary: it
     // is an ordinary launch, so everything earlier in the stream (e.g. the producer of X) has completed.
+    // PDL invariant: the fused kernel issues its TMA loads and bulk stores without griddepcontrol.wait, so it
+    // may only be a programmatic dependent of zero_checksums_kernel (which touches nothing but cs and waits
+    // for its own predecessor); pdl therefore requires d_cs, and the zero kernel is launched right before it.
     const bool pdl = d_cs && !(plan.flags & AOL_FLAG_NO_PDL);
     if (d_cs) {
         cudaLaunchConfig_t zc;

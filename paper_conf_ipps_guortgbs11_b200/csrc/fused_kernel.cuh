@@ -112,9 +112,6 @@ struct FusedArgs {
     uint32_t stage_stride;  // stage_bytes rounded up (1024 for the swizzle atom, 128 for uint8)
     uint32_t out_bytes;     // 4 output rows: 4 * Wo * sizeof(Tout)
     int32_t n_consumer;     // consumer threads, multiple of 32
-    int32_t hint_loads;     // 1: TMA loads with L2 evict_first (input is streamed once)
-    int32_t hint_stores;    // 1: bulk stores with L2 evict_first
-    int32_t blocked_units;  // 1: contiguous block of units per CTA instead of round-robin
     int32_t u8_tensor;      // uint8 path: 1 = 3-D TMA tensor loads (W % 128 == 0), 0 = 1-D bulk copies
     int32_t rows_per_stage; // int32 path: 3 (a stage holds a row triple) or 1 (one row per stage: finer ring
                             // granularity for wide frames); always 3 for uint8
@@ -127,19 +124,10 @@ __device__ __forceinline__ uint32_t swz(uint32_t line, uint32_t chunk) {
     return (line << 7) | (((chunk ^ line) & 7u) << 4);
 }
 
-// Same under SWIZZLE_32B for 32-byte lines (int32 frames with W % 32 != 0: one repetition = one line of
-// 8 elements): the 16-byte chunk index (0/1) XOR line bit 2 (address bit 4 ^= bit 7; 1024-aligned stages).
-// Eight consecutive lines then cover all eight 16-byte bank groups for either chunk: conflict-free LDS.128.
-__device__ __forceinline__ uint32_t swz32(uint32_t line, uint32_t chunk) {
-    return (line << 5) | (((chunk ^ (line >> 2)) & 1u) << 4);
-}
-
-// k-th work unit of this CTA: round-robin (concurrently running CTAs stream adjacent units) or, with
-// AOL_FLAG_BLOCKED_UNITS, a contiguous block of units per CTA.  Returns >= nunits when done.
-__device__ __forceinline__ int64_t unit_of(const FusedArgs& a, int64_t k) {
-    if (!a.blocked_units) return int64_t(blockIdx.x) + k * gridDim.x;
-    const int64_t per = (a.nunits + gridDim.x - 1) / gridDim.x;
-    return k < per ? int64_t(blockIdx.x) * per + k : a.nunits;
+// k-th work unit of this CTA: round-robin, so concurrently running CTAs stream adjacent units (a contiguous
+// block of units per CTA measured no faster, profiles/r01_blocked_units_ab.jsonl).  >= nunits when done.
+__device__ __forceinline__ int64_t unit_of(const FusedArgs&, int64_t k) {
+    return int64_t(blockIdx.x) + k * gridDim.x;
 }
 
 // Per-thread constants of the H stage (which repetition, where its bytes live).
@@ -147,7 +135,7 @@ struct RepGeom {
     uint32_t off0, off1;  // int32: swizzled offsets of the two chunks within a row's lines (kSwz = 0: byte
                           // offsets of the first / second chunk LOADED); uint8: 8r
     uint32_t offn;        // neighbour repetition's first chunk / word
-    uint32_t seg, segn;   // int32: 128-byte segment (32-byte line with kSwz == 32) of the repetition / neighbour
+    uint32_t seg, segn;   // int32: 128-byte segment of the repetition / neighbour
     bool fix;             // read the neighbour from smem instead of the shuffle
     bool swap;            // int32, kSwz = 0: the thread loads its upper chunk first (bank rotation)
 };
@@ -170,9 +158,6 @@ __device__ __forceinline__ void h_row(uint32_t row_base, uint32_t rr, const RepG
             const int4 B = ptx::lds128(rowa + g.off1);
             q0 = g.swap ? B : A;
             q1 = g.swap ? A : B;
-        } else if constexpr (kSwz == 32) {
-            q0 = ptx::lds128(row_base + swz32(line, 0));
-            q1 = ptx::lds128(row_base + swz32(line, 1));
         } else {
             q0 = ptx::lds128(row_base + swz(line, g.off0));
             q1 = ptx::lds128(row_base + swz(line, g.off1));
@@ -187,8 +172,6 @@ __device__ __forceinline__ void h_row(uint32_t row_base, uint32_t rr, const RepG
         int4 qn = q0;   // lane 31 / wrapping repetition: neighbour chunk from smem (predicated, no branch)
         if constexpr (kSwz == 0)
             ptx::lds128_if(qn, row_base + rr * (4u * W) + g.offn, g.fix);
-        else if constexpr (kSwz == 32)
-            ptx::lds128_if(qn, row_base + swz32(rr * segs + g.segn, 0), g.fix);
         else
             ptx::lds128_if(qn, row_base + swz(rr * segs + g.segn, g.offn), g.fix);
         dn = g.fix ? qn.x + qn.y + qn.z : dn;
@@ -259,9 +242,10 @@ __device__ __forceinline__ void h_row(uint32_t row_base, uint32_t rr, const RepG
 // kR = repetitions of the H tiler per consumer thread: 1 for int32 (two LDS.128 already cover one repetition's
 // 8 columns); 1 or 2 for uint8 input, whose 16 bytes for two repetitions come in one LDS.128 and whose per-stage
 // bookkeeping (mbarrier wait/arrive, addressing) two repetitions then share (the host picks, fused.cu).
-// kSwz = the int32 smem layout: 128 (TMA tensor loads under SWIZZLE_128B, W % 32 == 0), 0 (1-D bulk copies,
-// linear rows, any W % 8 == 0; the default when W % 32 != 0) or 32 (TMA tensor loads of 32-byte lines under
-// SWIZZLE_32B, W % 8 == 0 and W <= 2048; an A/B alternative to 0); unused (0) for uint8.  Tout = output element: int32, or int16 for 8-bit samples (outputs in [-5, 255]).
+// kSwz = the int32 smem layout: 128 (TMA tensor loads under SWIZZLE_128B, W % 32 == 0) or 0 (1-D bulk copies,
+// linear rows, any W % 8 == 0; the default when W % 32 != 0); 3 = packed 24-bit pixels; 0 for planar uint8.
+// (SWIZZLE_32B tensor lines for W % 32 != 0 measured no faster than linear rows and were removed,
+// profiles/r01_i32_layout_ab.jsonl.)  Tout = output element: int32, or int16 for 8-bit samples ([-5, 255]).
 template <typename Tin, typename Tout, int kR, int kSwz, bool kChecksum, int kMaxThreads, int kMinBlocks>
 __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
     fused_tma_kernel(const __grid_constant__ CUtensorMap tmap, const FusedArgs a) {
@@ -335,11 +319,7 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
                         const uint8_t* src = static_cast<const uint8_t*>(a.X) + size_t(row0 + 3 * trip) * 4u * a.W;
                         ptx::bulk_load(dst, src, a.stage_bytes, &full[s]);
                     } else if constexpr (kI32) {
-                        if (a.hint_loads)
-                            ptx::tma_load_3d_hint(dst, &tmap, &full[s], 0, 0, int32_t(row0 + 3 * trip),
-                                                  ptx::policy_evict_first());
-                        else
-                            ptx::tma_load_3d(dst, &tmap, &full[s], 0, 0, int32_t(row0 + 3 * trip));
+                        ptx::tma_load_3d(dst, &tmap, &full[s], 0, 0, int32_t(row0 + 3 * trip));
                     } else if (a.u8_tensor) {
                         // {128 B, W/128, rows} tensor, no swizzle: same linear smem layout as the bulk copy
                         ptx::tma_load_3d(dst, &tmap, &full[s], 0, 0, int32_t(row0 + 3 * trip));
@@ -371,10 +351,6 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
         g.off0 = 32u * uint32_t(r) + (g.swap ? 16u : 0u);
         g.off1 = 32u * uint32_t(r) + (g.swap ? 0u : 16u);
         g.offn = 32u * uint32_t(rn);
-    } else if constexpr (kI32 && kSwz == 32) {
-        g.seg = uint32_t(r);   // one 32-byte line per repetition
-        g.segn = uint32_t(rn);
-        g.off0 = g.off1 = g.offn = 0;
     } else if constexpr (kI32) {
         g.seg = uint32_t(r) >> 2;
         g.segn = uint32_t(rn) >> 2;
@@ -486,10 +462,7 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
             } else if (tid == 0) {
                 Tout* gz = static_cast<Tout*>(a.Z) + (size_t(plane) * a.Ho + size_t(4 * band)) * size_t(Wo);
                 const uint8_t* src = outbuf + (emit_idx % kOutBufs) * a.out_bytes;
-                if (a.hint_stores)
-                    ptx::bulk_store_hint(gz, src, a.out_bytes, ptx::policy_evict_first());
-                else
-                    ptx::bulk_store(gz, src, a.out_bytes);   // 4 rows
+                ptx::bulk_store(gz, src, a.out_bytes);   // 4 rows
                 ptx::bulk_commit();
             }
             ++emit_idx;
@@ -704,7 +677,7 @@ __global__ void __launch_bounds__(256)
 using KernelFn = void (*)(const CUtensorMap, const FusedArgs);
 
 // Explicit instantiations live in fused_k_*.cu (compiled in parallel); these pick one.
-KernelFn tma_kernel_i32(bool checksum, int layout, int block, int cps);   // layout = kSwz (128, 32 or 0)
+KernelFn tma_kernel_i32(bool checksum, int layout, int block, int cps);   // layout = kSwz (128 or 0)
 KernelFn tma_kernel_u8(bool checksum, bool out16, int reps_per_thread, int block, int cps);
 KernelFn tma_kernel_rgb8(bool checksum, bool out16, int block, int cps);   // packed 24-bit pixels
 

@@ -24,10 +24,14 @@ def built():
     _lib.lib()
 
 
+def header_text():
+    inc = os.path.join(ROOT, "include")
+    return "".join(open(os.path.join(inc, n)).read() for n in sorted(os.listdir(inc)) if n.endswith(".h"))
+
+
 def header_symbols():
-    with open(os.path.join(ROOT, "include", "aol.h")) as f:
-        text = f.read()
-    return sorted(set(re.findall(r"AOL_API\s+[\w\s\*]+?\b(aol_\w+)\s*\(", text)))
+    """Every entry point include/*.h declares (aol.h and the A/B-experiment header aol_tuning.h)."""
+    return sorted(set(re.findall(r"AOL_API\s+[\w\s\*]+?\b(aol_\w+)\s*\(", header_text())))
 
 
 def test_exports_every_declared_symbol():
@@ -233,13 +237,34 @@ def test_magic_division_formula():
         assert np.array_equal(q, xs // np.uint64(d)), d
 
 
+def test_headers_self_contained():
+    """include/aol.h and aol_tuning.h need only <stdint.h>/<stddef.h>: they compile as strict C99 with NO CUDA
+    include path (cudaStream_t is declared as cuda_runtime_api.h declares it), and as C++ together with the
+    CUDA runtime header in either order."""
+    import subprocess
+    import tempfile
+
+    d = tempfile.mkdtemp()
+    src = os.path.join(d, "h.c")
+    with open(src, "w") as f:
+        f.write('#include "aol_tuning.h"\nint main(void) { cudaStream_t s = 0; (void)s; return aol_version() != AOL_VERSION; }\n')
+    subprocess.check_call(["gcc", "-std=c99", "-pedantic", "-Wall", "-Wextra", "-Werror", "-I",
+                           os.path.join(ROOT, "include"), "-c", src, "-o", os.path.join(d, "h.o")])
+    for first, second in (("aol.h", "cuda_runtime_api.h"), ("cuda_runtime_api.h", "aol.h")):
+        cpp = os.path.join(d, "h.cpp")
+        with open(cpp, "w") as f:
+            f.write(f'#include "{first}"\n#include "{second}"\nint g() {{ return aol_version(); }}\n')
+        subprocess.check_call(["g++", "-std=c++11", "-Wall", "-Werror", "-I", os.path.join(ROOT, "include"), "-I",
+                               "/usr/local/cuda/include", "-c", cpp, "-o", os.path.join(d, "h2.o")])
+
+
 def test_c_example_builds_against_header():
-    """examples/aol_example.c compiles and links against include/aol.h + libaol.so with gcc (C99)."""
+    """examples/aol_example.c compiles and links against include/aol.h + libaol.so with gcc (C11)."""
     import subprocess
     import tempfile
 
     out = os.path.join(tempfile.mkdtemp(), "aol_example")
-    subprocess.check_call(["gcc", "-std=c99", "-O2", "-Wall", "-Wextra", "-Werror", "-I", os.path.join(ROOT, "include"),
+    subprocess.check_call(["gcc", "-std=c11", "-O2", "-Wall", "-Wextra", "-Werror", "-I", os.path.join(ROOT, "include"),
                            "-I", "/usr/local/cuda/include", os.path.join(ROOT, "examples", "aol_example.c"),
                            "-L", os.path.dirname(_lib.LIB_PATH), "-laol", "-L", "/usr/local/cuda/lib64", "-lcudart",
                            "-o", out])
@@ -251,7 +276,7 @@ def test_binding_constants_match_header():
     a drifted constant would silently select another dtype, preset or launch option)."""
     import re
 
-    hdr = open(os.path.join(ROOT, "include", "aol.h")).read()
+    hdr = header_text()
     flags = {m.group(1): int(m.group(2)) for m in re.finditer(r"#define AOL_FLAG_(\w+)\s+(\d+)", hdr)}
     assert flags == aol.FLAGS
     for name, val in (("AOL_U8", _lib.U8), ("AOL_I16", _lib.I16), ("AOL_I32", _lib.I32), ("AOL_I64", _lib.I64),

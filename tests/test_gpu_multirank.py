@@ -53,7 +53,7 @@ def test_weak_two_ranks(orc, tmp_path):
 def test_strong_stream_two_ranks(orc, tmp_path):
     # 23 stream frames: rank 0 owns global frames 0..11, rank 1 owns 12..22; pools of 4 frames per rank
     d, cs = run2(tmp_path, "--stream-frames", "23", "--pool", "4")
-    assert d["scaling"] == "strong" and d["config"]["launches_per_step"] == 3 and d["gpu_launches"] == 18
+    assert d["scaling"] == "strong" and d["launch"]["launches_per_step"] == 3 and d["gpu_launches"] == 18
     _, ref0 = orc.downscale_frame(synth.frames(0, 0, 4, C, H, W), nthreads=8)
     _, ref1 = orc.downscale_frame(synth.frames(0, 12, 4, C, H, W), nthreads=8)
     assert np.array_equal(cs, np.concatenate([ref0, ref1]))

@@ -5,6 +5,8 @@ The arithmetic is integer (Fig. 5, SaC `int`), so the bar is exact equality
 synth/ (numpy) for the oracle side; the GPU side receives the same arrays, or
 generates them with its own counter-based generator (checked equal first).
 """
+import os
+
 import numpy as np
 import pytest
 import torch
@@ -79,8 +81,8 @@ def test_fused_vs_oracle(orc, shape, kernel):
 @pytest.mark.parametrize("opts", [
     {"bands_per_unit": 1}, {"bands_per_unit": 2}, {"bands_per_unit": 7}, {"bands_per_unit": 40},
     {"stages": 2}, {"stages": 3, "bands_per_unit": 5}, {"ctas_per_sm": 2}, {"ctas_per_sm": 2, "stages": 2},
-    {"flags": 8}, {"flags": 8, "bands_per_unit": 1, "stages": 2}, {"ctas_per_sm": 4}, {"ctas_per_sm": 8, "stages": 2},
-    {"flags": 2}, {"flags": 4},
+    {"flags": 64}, {"flags": 64, "bands_per_unit": 1, "stages": 2}, {"ctas_per_sm": 4}, {"ctas_per_sm": 8, "stages": 2},
+    {"flags": 128}, {"flags": 1024},
 ])
 def test_fused_launch_options(orc, opts):
     """Unit boundaries, ring wrap-around and CTA residency do not change results."""
@@ -101,15 +103,15 @@ def test_fused_launch_options(orc, opts):
                                    (1, 3, 18, 24), (2, 1, 27, 1448)])
 def test_unaligned_width_shapes(orc, shape):
     """int32, W % 32 != 0 (e.g. 720-wide SD frames): the TMA kernel on linear rows (1-D bulk copies of the
-    row triple, lane-rotated LDS.128; the default), on 32-byte lines under SWIZZLE_32B (AOL_FLAG_I32_SWZ32 =
-    256, W <= 2048), against the oracle and the generic kernel, with and without checksums."""
+    row triple, lane-rotated LDS.128), against the oracle and the generic kernel, with and without
+    checksums."""
     N, C, H, W = shape
     xh = synth.frames(5, 0, N, C, H, W, "signed")
     zo, cso = run_oracle(orc, xh)
     assert aol.downscale_frame_plan(N, C, H, W)["kernel"] == 1
     x = torch.from_numpy(xh).cuda()
-    for opts in (None, {"kernel": 1, "ctas_per_sm": 2, "bands_per_unit": 1}, {"kernel": 1, "flags": 256},
-                 {"kernel": 1, "flags": 256, "ctas_per_sm": 3, "stages": 2}, {"kernel": 2}):
+    for opts in (None, {"kernel": 1, "ctas_per_sm": 2, "bands_per_unit": 1},
+                 {"kernel": 1, "ctas_per_sm": 3, "stages": 2}, {"kernel": 2}):
         z, cs = aol.downscale_frame(x, checksums=True, opts=opts)
         z2, _ = aol.downscale_frame(x, opts=opts)
         torch.cuda.synchronize()
@@ -158,21 +160,22 @@ def test_linear_rows_forced(orc, shape):
 
 @pytest.mark.parametrize("shape", [(1, 1, 9, 2056), (1, 2, 18, 4008), (1, 1, 9, 7432)])
 def test_wide_unaligned_shapes(orc, shape):
-    """int32, W % 32 != 0 and W > 2048: linear rows (a TMA box dimension holds <= 256 lines, so the
-    SWIZZLE_32B layout cannot take these widths and falls back to the generic fused kernel)."""
+    """int32, W % 32 != 0 and W > 2048: linear rows (one-row ring stages beyond W = 3271), against the
+    oracle and the generic fused kernel; unknown flag bits (the removed SWIZZLE_32B layout's 256) are refused."""
     N, C, H, W = shape
     xh = synth.frames(5, 0, N, C, H, W, "signed")
     zo, cso = run_oracle(orc, xh)
     assert aol.downscale_frame_plan(N, C, H, W)["kernel"] == 1
-    assert aol.downscale_frame_plan(N, C, H, W, opts={"flags": 256})["kernel"] == 2
     x = torch.from_numpy(xh).cuda()
-    for opts in (None, {"flags": 256}):
+    for opts in (None, {"kernel": 2}):
         z, cs = aol.downscale_frame(x, checksums=True, opts=opts)
         torch.cuda.synchronize()
         assert np.array_equal(z.cpu().numpy(), zo), opts
         assert np.array_equal(np_u64(cs), cso), opts
     with pytest.raises(aol.AolError):
         aol.downscale_frame(x, opts={"kernel": 1, "flags": 256})
+    with pytest.raises(aol.AolError):
+        aol.downscale_frame_plan(N, C, H, W, opts={"flags": 2})
 
 
 @pytest.mark.parametrize("shape,kernel", [
@@ -200,8 +203,8 @@ def test_fused_u8_launch_options(orc):
     xh = synth.frames(22, 0, 3, 3, 117, 512, "uniform")
     zo, cso = run_oracle(orc, xh)
     x8 = torch.from_numpy(xh.astype(np.uint8)).cuda()
-    for o in ({"bands_per_unit": 1}, {"stages": 2}, {"ctas_per_sm": 2}, {"ctas_per_sm": 4}, {"flags": 16},
-              {"flags": 24, "bands_per_unit": 3}):
+    for o in ({"bands_per_unit": 1}, {"stages": 2}, {"ctas_per_sm": 2}, {"ctas_per_sm": 4}, {"flags": 64},
+              {"flags": 96, "bands_per_unit": 3}):
         z, cs = aol.downscale_frame(x8, checksums=True, opts=dict(o, kernel=1))
         torch.cuda.synchronize()
         assert np.array_equal(z.cpu().numpy(), zo), o
@@ -219,7 +222,7 @@ def test_fused_u8_two_reps_per_thread(orc, W):
     xh[0, 1] = synth.frames(24, 0, 1, 1, H, W, "dark")[0, 0]   # negative V sums on one plane
     zo, cso = run_oracle(orc, xh)
     x8 = torch.from_numpy(xh.astype(np.uint8)).cuda()
-    for flags in (0, 32, 16):
+    for flags in (0, 32, 64):
         o = {"kernel": 1, "flags": flags}
         plan = aol.downscale_frame_plan(N, C, H, W, dtype=torch.uint8, opts=o)
         z, cs = aol.downscale_frame(x8, checksums=True, opts=o)
@@ -510,10 +513,22 @@ def test_tiler_batch_descriptor(orc):
 
 # -------------------------------------------------------------- full-size configs
 
+def _oracle_cs(orc, seed, index, C, H, W, chunk=16):
+    """Oracle checksums of synthetic frames `index` (global frame indices), generated in chunks by the C form
+    of the seeded generator."""
+    index = list(index)
+    out = np.empty(len(index), np.uint64)
+    for k in range(0, len(index), chunk):
+        idx = index[k:k + chunk]
+        _, cs = orc.downscale_frame(synth.frames_c(seed, 0, len(idx), C, H, W, index=idx), nthreads=16)
+        out[k:k + len(idx)] = cs
+    return out
+
+
 def test_bench_config_300_hd_frames(orc):
-    """BASELINE configs[1]: 300 HD frames, the launch bench.py times.  Sampled frames are
-    compared element by element with the oracle; every frame's fused checksum must equal
-    the stand-alone checksum kernel, and sampled checksums the oracle's."""
+    """BASELINE configs[1]: 300 HD frames, the launch bench.py times.  EVERY frame's checksum against the
+    oracle; frames {0, 149, 299} element by element; the fused epilogue against the
+    stand-alone checksum kernel."""
     N, C, H, W = 300, 3, 1080, 1920
     x = aol.synth_frames(0, 0, N, C, H, W, "uniform")
     z, cs = aol.downscale_frame(x, checksums=True)
@@ -526,17 +541,15 @@ def test_bench_config_300_hd_frames(orc):
         zo, cso = run_oracle(orc, xh)
         assert np.array_equal(z[n:n + 1].cpu().numpy(), zo), n
         assert np_u64(cs[n:n + 1])[0] == cso[0]
-    # checksums of a spread of further frames (every 25th) against the oracle
     got = np_u64(cs)
-    for n in range(12, 300, 25):
-        _, cso = run_oracle(orc, synth.frames(0, n, 1, C, H, W, "uniform"))
-        assert got[n] == cso[0], n
+    want = _oracle_cs(orc, 0, range(N), C, H, W)
+    bad = np.nonzero(got != want)[0]
+    assert bad.size == 0, f"{bad.size} of 300 frame checksums differ from the oracle, first {bad[:8]}"
 
 
 def test_4k_batch(orc):
-    """BASELINE configs[3]: the 64-frame 3840x2160 batch tools/bench_configs.py times.
-    Frames {0, 63} element by element against the oracle; every frame's fused checksum against the
-    stand-alone checksum kernel; a spread of checksums against the oracle."""
+    """BASELINE configs[3]: the 64-frame 3840x2160 batch bench.py's d4 record times.
+    EVERY frame's checksum against the oracle; frames {0, 63} element by element."""
     N, C, H, W = 64, 3, 2160, 3840
     x = aol.synth_frames(1, 0, N, C, H, W, "uniform")
     z, cs = aol.downscale_frame(x, checksums=True)
@@ -548,11 +561,28 @@ def test_4k_batch(orc):
         zo, cso = run_oracle(orc, synth.frames(1, n, 1, C, H, W, "uniform"))
         assert np.array_equal(z[n:n + 1].cpu().numpy(), zo)
         assert got[n] == cso[0]
-    for n in range(7, N - 1, 14):
-        _, cso = run_oracle(orc, synth.frames(1, n, 1, C, H, W, "uniform"))
-        assert got[n] == cso[0], n
     del x, z
     torch.cuda.empty_cache()
+    assert np.array_equal(got, _oracle_cs(orc, 1, range(N), C, H, W))
+
+
+def test_d5_hd_stream_pool_512_frames(orc, tmp_path):
+    """SURVEY 8(d) d5 at full HD size: a 512-frame stream through bench.py's strong-scaling mode with a device
+    pool of 256 frames (two launches over the pool); the pool's 256 checksums against the oracle."""
+    import json
+    import subprocess
+    import sys
+
+    from conftest import ROOT
+
+    dump = str(tmp_path / "cs.npy")
+    r = subprocess.run([sys.executable, os.path.join(ROOT, "bench.py"), "--stream-frames", "512", "--pool", "256",
+                        "--steps", "3", "--warmup", "3", "--no-cpu-baseline", "--dump-checksums", dump],
+                       capture_output=True, text=True, timeout=900, cwd=ROOT)
+    assert r.returncode == 0, r.stderr[-3000:]
+    d = json.loads([l for l in r.stdout.splitlines() if l.startswith("{")][-1])
+    assert d["scaling"] == "strong" and d["launch"]["launches_per_step"] == 2
+    assert np.array_equal(np.load(dump), _oracle_cs(orc, 0, range(256), 3, 1080, 1920))
 
 
 def test_cif_2000_frames(orc):
@@ -795,3 +825,66 @@ def test_packed_rgb_host_streamed(orc):
     zo, cso = run_oracle(orc, xp)
     assert np.array_equal(z.numpy(), zo)
     assert np.array_equal(cs.view(torch.int64).numpy().view(np.uint64), cso)
+
+
+@pytest.mark.parametrize("W,out_dtype,ok", [(6400, torch.int32, True), (6416, torch.int32, False),
+                                            (6416, torch.int16, True), (7936, torch.int16, True)])
+def test_packed_rgb_width_limit(orc, W, out_dtype, ok):
+    """Packed 24-bit pixels: two 9W-byte ring stages plus the 3-plane output staging (18W bytes int32, 9W int16)
+    fit the 227 KB opt-in up to W = 6400 with int32 outputs and W = 7936 with int16 outputs; the first width past
+    the int32 limit is refused with a message naming that limit."""
+    N, H = 1, 9
+    xp = synth.frames(25, 0, N, 3, H, W, "uniform")
+    packed = torch.from_numpy(np.ascontiguousarray(np.transpose(xp, (0, 2, 3, 1))).astype(np.uint8)).cuda()
+    if not ok:
+        with pytest.raises(aol.AolError) as e:
+            aol.downscale_frame_packed(packed, out_dtype=out_dtype)
+        assert e.value.status == aol._lib.E_SHAPE and "W <= 6400 with int32" in str(e.value)
+        return
+    z, cs = aol.downscale_frame_packed(packed, checksums=True, out_dtype=out_dtype)
+    zo, cso = run_oracle(orc, xp)
+    torch.cuda.synchronize()
+    assert np.array_equal(z.cpu().numpy().astype(np.int32), zo) and np.array_equal(np_u64(cs), cso)
+
+
+@pytest.mark.parametrize("kernel", [1, 2])
+def test_failed_launch_enqueues_nothing(kernel):
+    """A call that fails at its launch (forced by the test hook right before the first enqueue) returns
+    AOL_E_CUDA and leaves the caller's output and checksum buffers untouched (include/aol.h: on error nothing
+    has been enqueued); the next call works."""
+    import ctypes
+
+    N, C, H, W = 2, 3, 36, 128
+    x = aol.synth_frames(3, 0, N, C, H, W)
+    z = torch.full((N, C, 16, 48), -77, dtype=torch.int32, device="cuda")
+    cs = torch.full((N,), 12345, dtype=torch.int64, device="cuda").view(torch.uint64)
+    aol._lib.lib().aol_debug_fail_next_launches(1)
+    with pytest.raises(aol.AolError) as e:
+        aol.downscale_frame(x, out=z, checksums=cs, opts={"kernel": kernel})
+    assert e.value.status == aol._lib.E_CUDA and "injected" in str(e.value)
+    torch.cuda.synchronize()
+    assert bool((z == -77).all()) and bool((cs.view(torch.int64) == 12345).all())
+    aol.downscale_frame(x, out=z, checksums=cs, opts={"kernel": kernel})
+    torch.cuda.synchronize()
+    assert not bool((z == -77).any()) and not bool((cs.view(torch.int64) == 12345).any())
+
+
+def test_misaligned_checksum_pointer_refused():
+    """d_frame_checksums must be 8-byte aligned (a misaligned u64 atomic would be a sticky context fault):
+    AOL_E_ALIGN from the fused call and from aol_frame_checksum, through the C ABI with raw pointers."""
+    import ctypes
+
+    L = aol._lib.lib()
+    N, C, H, W = 1, 3, 18, 64
+    x = aol.synth_frames(3, 0, N, C, H, W)
+    z = torch.empty((N, C, 8, 24), dtype=torch.int32, device="cuda")
+    buf = torch.zeros(4, dtype=torch.int64, device="cuda")
+    bad = ctypes.c_void_p(buf.data_ptr() + 4)
+    st = L.aol_downscale_frame(ctypes.c_void_p(x.data_ptr()), aol._lib.I32, ctypes.c_void_p(z.data_ptr()), N, C, H, W,
+                               bad, ctypes.c_void_p(torch.cuda.current_stream().cuda_stream))
+    assert st == aol._lib.E_ALIGN
+    st = L.aol_frame_checksum(ctypes.c_void_p(z.data_ptr()), N, C, 8, 24, bad,
+                              ctypes.c_void_p(torch.cuda.current_stream().cuda_stream))
+    assert st == aol._lib.E_ALIGN
+    torch.cuda.synchronize()
+    assert bool((buf == 0).all())

@@ -31,3 +31,19 @@ def test_ranges():
     assert np.array_equal(r[0, 1, 2], np.arange(40))
     c = synth.frames(1, 0, 1, 1, 2, 8, "constant", value=-9)
     assert np.all(c == -9)
+
+
+def test_c_generator_equals_numpy():
+    """synth.c (OpenMP, used for bench-size oracle inputs) produces the numpy generator's frames bit for bit,
+    for every kind, both element types, a seed above 2^63 and an explicit global-frame index list."""
+    for kind in synth.KINDS:
+        for seed in (0, 7, (1 << 64) - 3):
+            a = synth.frames(seed, 3, 2, 3, 9, 24, kind, value=-5)
+            b = synth.frames_c(seed, 3, 2, 3, 9, 24, kind, value=-5)
+            assert np.array_equal(a, b), (kind, seed)
+    u = synth.frames_c(11, 0, 2, 3, 9, 32, "uniform", dtype=np.uint8)
+    assert u.dtype == np.uint8 and np.array_equal(u.astype(np.int32), synth.frames(11, 0, 2, 3, 9, 32))
+    idx = [5, 0, 257, 5]
+    c = synth.frames_c(2, 0, 4, 3, 9, 16, index=idx)
+    for n, g in enumerate(idx):
+        assert np.array_equal(c[n], synth.frames(2, g, 1, 3, 9, 16)[0])

@@ -37,7 +37,7 @@ def main():
             x = aol.synth_frames(1, 0, N, C, H, W, "uniform", dtype=dt)
             ref = None
             all_opts = [{"kernel": 2}, {"kernel": 1}, {"kernel": 1, "stages": 2, "bands_per_unit": 1},
-                        {"kernel": 1, "ctas_per_sm": 2}, {"kernel": 1, "flags": 8}]
+                        {"kernel": 1, "ctas_per_sm": 2}, {"kernel": 1, "flags": 64}]
             for opts in [o for o in all_opts if o["kernel"] in kernels]:
                 try:
                     z, cs = aol.downscale_frame(x, checksums=True, opts=opts)
