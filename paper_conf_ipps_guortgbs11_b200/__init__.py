@@ -152,8 +152,8 @@ def tiler_scatter(t: aol_tiler_t, tiles: torch.Tensor, array: torch.Tensor, mode
     _out(tiles, rep + pat, array.dtype, array.device, "tiles")
     m = {"fast": SCATTER_FAST, "sequential": SCATTER_SEQUENTIAL}[mode]
     ws_ptr, ws_bytes = ctypes.c_void_p(0), 0
-    if m == SCATTER_SEQUENTIAL:
-        need = int(lib().aol_tiler_scatter_workspace_bytes(ctypes.byref(t)))
+    need = int(lib().aol_tiler_scatter_workspace_bytes(ctypes.byref(t))) if m == SCATTER_SEQUENTIAL else 0
+    if need > 0:   # 0: the library proved the tiler injective (no claims needed) or the mode is FAST
         if workspace is None:
             workspace = torch.empty(need, dtype=torch.uint8, device=array.device)
         if workspace.device != array.device:

@@ -172,7 +172,50 @@ aol_status_t validate_tiler(const aol_tiler_t* t) {
     return AOL_OK;
 }
 
+// A sufficient condition for injectivity of (r, i) -> (o + P.r + F.i) mod s, checked on the host in
+// O(rank^2): every combined (repetition or pattern) dim d with extent > 1 moves exactly ONE array dim a(d),
+// with signed coefficient c_d (the representative of c mod s_a nearest 0); per array dim, the coefficients
+// of its dims, sorted by |c|, dominate (|c_d| > sum over smaller ones of |c_e| (ext_e - 1): mixed-radix
+// digits, so distinct index vectors give distinct raw coordinates), and the raw coordinates span at most
+// s_a values (so the modulo keeps them distinct).  The paper's output tilers, blockings and their wrapping
+// variants qualify; anything it cannot prove takes the two-pass claim path.
+bool prove_injective(const TilerDev& td) {
+    int owner[2 * AOL_MAX_RANK];
+    int64_t sc[2 * AOL_MAX_RANK];
+    for (int d = 0; d < td.nd; ++d) {
+        owner[d] = -1;
+        if (td.ext[d] == 1) continue;
+        for (int a = 0; a < td.ra; ++a) {
+            int64_t c = td.coef[a][d];
+            if (c == 0) continue;
+            if (owner[d] >= 0) return false;   // moves two array dims: not provable here
+            if (2 * c > td.ashape[a]) c -= td.ashape[a];
+            owner[d] = a;
+            sc[d] = c < 0 ? -c : c;
+        }
+        if (owner[d] < 0) return false;         // broadcast dim: two indices hit the same element
+    }
+    for (int a = 0; a < td.ra; ++a) {
+        int ds[2 * AOL_MAX_RANK], n = 0;
+        for (int d = 0; d < td.nd; ++d)
+            if (td.ext[d] > 1 && owner[d] == a) ds[n++] = d;
+        std::sort(ds, ds + n, [&](int x, int y) { return sc[x] < sc[y]; });
+        __int128 acc = 0;   // largest |raw offset| the smaller digits reach
+        for (int k = 0; k < n; ++k) {
+            if (__int128(sc[ds[k]]) <= acc) return false;
+            acc += __int128(sc[ds[k]]) * (td.ext[ds[k]] - 1);
+        }
+        if (acc + 1 > td.ashape[a]) return false;
+    }
+    return true;
+}
+
 }  // namespace
+
+int claim_bytes(const TilerDev& td) {
+    if (td.proven_injective) return 0;
+    return td.total < (int64_t(1) << 32) - 1 ? 4 : 8;
+}
 
 aol_status_t make_tiler_dev(const aol_tiler_t* t, TilerDev* td) {
     aol_status_t st = validate_tiler(t);
@@ -260,6 +303,7 @@ aol_status_t make_tiler_dev(const aol_tiler_t* t, TilerDev* td) {
         td->p_fd_mul[i] = td->fd_mul[d];
         td->p_fd_shift[i] = td->fd_shift[d];
     }
+    td->proven_injective = prove_injective(*td) ? 1 : 0;
     return AOL_OK;
 }
 
@@ -386,6 +430,10 @@ aol_status_t aol_tiler_is_injective(const aol_tiler_t* t, int* injective) {
     TilerDev td;
     aol_status_t st = make_tiler_dev(t, &td);
     if (st != AOL_OK) return st;
+    if (td.proven_injective) {   // the host proof (prove_injective) is sound: no enumeration needed
+        *injective = 1;
+        return AOL_OK;
+    }
     if (td.array_elems > (int64_t(1) << 32) || td.total > (int64_t(1) << 32))
         return fail(AOL_E_RANGE, "brute-force injectivity check limited to 2^32 elements");
     std::vector<uint64_t> seen;   // one bit per array element (<= 512 MiB)
@@ -433,7 +481,7 @@ aol_status_t aol_tiler_gather(const aol_tiler_t* t, aol_dtype_t el, const void* 
 size_t aol_tiler_scatter_workspace_bytes(const aol_tiler_t* t) {
     TilerDev td;
     if (make_tiler_dev(t, &td) != AOL_OK) return 0;
-    return size_t(td.array_elems) * 8;
+    return size_t(td.array_elems) * size_t(claim_bytes(td));
 }
 
 aol_status_t aol_tiler_scatter(const aol_tiler_t* t, aol_dtype_t el, const void* d_tiles, void* d_array,
@@ -447,8 +495,8 @@ aol_status_t aol_tiler_scatter(const aol_tiler_t* t, aol_dtype_t el, const void*
     if ((reinterpret_cast<uintptr_t>(d_array) | reinterpret_cast<uintptr_t>(d_tiles)) % es)
         return fail(AOL_E_ALIGN, "buffers must be aligned to the element size");
     if (mode != AOL_SCATTER_FAST && mode != AOL_SCATTER_SEQUENTIAL) return fail(AOL_E_INVALID, "bad scatter mode");
-    if (mode == AOL_SCATTER_SEQUENTIAL) {
-        if (!d_workspace || ws_bytes < size_t(td.array_elems) * 8)
+    if (mode == AOL_SCATTER_SEQUENTIAL && claim_bytes(td) > 0) {
+        if (!d_workspace || ws_bytes < size_t(td.array_elems) * size_t(claim_bytes(td)))
             return fail(AOL_E_WORKSPACE, "SEQUENTIAL scatter needs aol_tiler_scatter_workspace_bytes() of workspace");
         if (reinterpret_cast<uintptr_t>(d_workspace) % 8) return fail(AOL_E_ALIGN, "workspace must be 8-byte aligned");
     }

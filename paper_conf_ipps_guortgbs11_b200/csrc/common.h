@@ -102,7 +102,12 @@ struct TilerDev {
     uint32_t p_fd_mul[2 * AOL_MAX_RANK], p_fd_shift[2 * AOL_MAX_RANK];
     int64_t total;              // rep elements * pattern elements
     int64_t array_elems;
+    int32_t proven_injective;   // 1: the host proved no two (r, i) address the same element (see api.cu);
+                                // SEQUENTIAL scatters then take the one-pass FAST kernels
 };
+// Bytes per array element of the SEQUENTIAL scatter's claim workspace: 0 when proven injective, 4 when every
+// claim (flat tile index + 1) fits 32 bits, else 8.
+int claim_bytes(const TilerDev& td);
 aol_status_t make_tiler_dev(const aol_tiler_t* t, TilerDev* out);
 aol_status_t launch_gather(const TilerDev& td, int elsize, const void* d_array, void* d_tiles, cudaStream_t s);
 aol_status_t launch_scatter(const TilerDev& td, int elsize, const void* d_tiles, void* d_array, int sequential,

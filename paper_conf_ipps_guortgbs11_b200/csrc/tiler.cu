@@ -25,7 +25,8 @@
 
 namespace aol {
 
-// per-element-size launchers (tiler_es{1,2,4,8}.cu); mode 0 gather, 1 FAST scatter, 2/3 SEQUENTIAL passes
+// per-element-size launchers (tiler_es{1,2,4,8}.cu); mode 0 gather, 1 FAST scatter, 2/3 SEQUENTIAL passes with
+// 8-byte claims, 4/5 the same with 4-byte claims
 aol_status_t tiler_launch_es1(int mode, const TilerDev& td, int vec, const void* src, void* dst,
                               unsigned long long* ws, int num_sms, cudaStream_t s);
 aol_status_t tiler_launch_es2(int mode, const TilerDev& td, int vec, const void* src, void* dst,
@@ -83,13 +84,20 @@ aol_status_t launch_scatter(const TilerDev& td, int elsize, const void* d_tiles,
     aol_status_t st = device_info(&dev);
     if (st != AOL_OK) return st;
     auto* ws = static_cast<unsigned long long*>(d_ws);
-    if (!sequential)
+    // a SEQUENTIAL scatter whose tiler the host proved injective has no collisions: Fig. 6's loop order cannot
+    // change the result, so it takes the one-pass FAST kernels (no workspace)
+    const int cb = claim_bytes(td);
+    if (!sequential || cb == 0)
         return launch_mode<1>(td, elsize, vector_width(td, elsize, d_array, d_tiles), d_tiles, d_array, nullptr,
                               dev.num_sms, s);
-    AOL_CUDA_TRY(cudaMemsetAsync(d_ws, 0, size_t(td.array_elems) * 8, s));
-    st = launch_mode<2>(td, elsize, 1, d_tiles, d_array, ws, dev.num_sms, s);
+    // two passes: claim (the largest flat tile index + 1 per target: the last writer in Fig. 6 order), then
+    // write where this element holds the claim; 4-byte claims when every claim fits 32 bits
+    AOL_CUDA_TRY(cudaMemsetAsync(d_ws, 0, size_t(td.array_elems) * size_t(cb), s));
+    st = cb == 4 ? launch_mode<4>(td, elsize, 1, d_tiles, d_array, ws, dev.num_sms, s)
+                 : launch_mode<2>(td, elsize, 1, d_tiles, d_array, ws, dev.num_sms, s);
     if (st != AOL_OK) return st;
-    return launch_mode<3>(td, elsize, 1, d_tiles, d_array, ws, dev.num_sms, s);
+    return cb == 4 ? launch_mode<5>(td, elsize, 1, d_tiles, d_array, ws, dev.num_sms, s)
+                   : launch_mode<3>(td, elsize, 1, d_tiles, d_array, ws, dev.num_sms, s);
 }
 
 }  // namespace aol

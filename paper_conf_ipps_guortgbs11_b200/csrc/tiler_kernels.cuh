@@ -117,7 +117,19 @@ __device__ __forceinline__ int64_t general_offset(const TilerDev& td, const int6
 }
 
 // mode 0: gather; 1: FAST scatter; 2: SEQUENTIAL claim (max flat index + 1 per target);
-// 3: SEQUENTIAL write (store iff this element holds the claim).
+// 3: SEQUENTIAL write (store iff this element holds the claim); 4 / 5: the same with 4-byte claims.
+template <int MODE>
+__device__ __forceinline__ void seq_pass(void* ws, int64_t off, int64_t g, bool& write) {
+    if constexpr (MODE == 2) {
+        atomicMax(static_cast<unsigned long long*>(ws) + off, (unsigned long long)g + 1ull);
+    } else if constexpr (MODE == 4) {
+        atomicMax(static_cast<unsigned int*>(ws) + off, unsigned(g) + 1u);
+    } else if constexpr (MODE == 3) {
+        write = static_cast<const unsigned long long*>(ws)[off] == (unsigned long long)g + 1ull;
+    } else if constexpr (MODE == 5) {
+        write = static_cast<const unsigned int*>(ws)[off] == unsigned(g) + 1u;
+    }
+}
 template <int ES, int V, bool kFast32, bool kLinear, int MODE>
 __global__ void __launch_bounds__(256) tiler_kernel(const TilerDev td, const void* __restrict__ src,
                                                     void* __restrict__ dst, unsigned long long* __restrict__ ws) {
@@ -186,11 +198,10 @@ __global__ void __launch_bounds__(256) tiler_kernel(const TilerDev td, const voi
 #pragma unroll
             for (int u = 0; u < kU; ++u)
                 if (v0 + 32 * u < nvec) reinterpret_cast<VT*>(static_cast<T*>(dst) + off[u])[0] = val[u];
-        } else if (MODE == 2) {
-            atomicMax(ws + off[0], (unsigned long long)g[0] + 1ull);
-        } else {
-            if (ws[off[0]] == (unsigned long long)g[0] + 1ull)
-                static_cast<T*>(dst)[off[0]] = static_cast<const T*>(src)[g[0]];
+        } else if (v0 < nvec) {   // SEQUENTIAL passes (V == 1, kU == 1)
+            bool write = false;
+            seq_pass<MODE>(ws, off[0], g[0], write);
+            if (write) static_cast<T*>(dst)[off[0]] = static_cast<const T*>(src)[g[0]];
         }
     }
 }
@@ -327,11 +338,10 @@ __global__ void __launch_bounds__(256) tiler_wrap32_kernel(const Wrap32Dev wd, c
 #pragma unroll
             for (int u = 0; u < kU; ++u)
                 if (g[u] < n_el) static_cast<T*>(dst)[off[u]] = val[u];
-        } else if (MODE == 2) {   // SEQUENTIAL claim: the last (r, i) in row-major order wins
-            if (g[0] < n_el) atomicMax(ws + off[0], (unsigned long long)g[0] + 1ull);
-        } else {                  // SEQUENTIAL write
-            if (g[0] < n_el && ws[off[0]] == (unsigned long long)g[0] + 1ull)
-                static_cast<T*>(dst)[off[0]] = static_cast<const T*>(src)[g[0]];
+        } else if (g[0] < n_el) {   // SEQUENTIAL claim / write: the last (r, i) in row-major order wins
+            bool write = false;
+            seq_pass<MODE>(ws, off[0], g[0], write);
+            if (write) static_cast<T*>(dst)[off[0]] = static_cast<const T*>(src)[g[0]];
         }
     }
 }

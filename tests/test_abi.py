@@ -122,9 +122,47 @@ def test_paper_tilers_injectivity():
     assert not aol.tiler_is_injective(aol.tiler_preset(aol.PRESET_V_IN, 18, 24))
 
 
+@pytest.mark.parametrize("seed", range(400))
+def test_injectivity_proof_is_sound(seed):
+    """The host's injectivity proof (SEQUENTIAL scatters of proven tilers take the one-pass FAST kernels and
+    need no workspace) never claims a tiler the brute-force enumeration finds non-injective."""
+    rng = np.random.default_rng(5000 + seed)
+    d = bf.random_descriptor(rng)
+    if seed % 2:   # bias half the cases toward block-diagonal (provable) descriptors
+        ra, rr, rp = len(d["array_shape"]), len(d["rep_shape"]), len(d["pattern_shape"])
+        for j in range(rr):
+            a = int(rng.integers(ra))
+            for b in range(ra):
+                d["paving"][b][j] = int(rng.integers(-9, 10)) if b == a else 0
+        for k in range(rp):
+            a = int(rng.integers(ra))
+            for b in range(ra):
+                d["fitting"][b][k] = int(rng.integers(-3, 4)) if b == a else 0
+    t = aol.make_tiler(d["array_shape"], d["rep_shape"], d["pattern_shape"], d["origin"], d["paving"], d["fitting"])
+    proven = _lib.lib().aol_tiler_scatter_workspace_bytes(ctypes.byref(t)) == 0
+    cnt = bf.read_counts(d["array_shape"], d["rep_shape"], d["pattern_shape"], d["origin"], d["paving"],
+                         d["fitting"])
+    if proven:
+        assert cnt.max() <= 1, d
+    assert aol.tiler_is_injective(t) == bool(cnt.max() <= 1)
+
+
+def test_injectivity_proof_covers_the_paper_and_d3_tilers():
+    L = _lib.lib()
+    ws = lambda t: L.aol_tiler_scatter_workspace_bytes(ctypes.byref(t))  # noqa: E731
+    assert ws(aol.tiler_preset(aol.PRESET_H_OUT, 18, 64)) == 0 and ws(aol.tiler_preset(aol.PRESET_V_OUT, 18, 24)) == 0
+    assert ws(aol.tiler_preset(aol.PRESET_H_IN, 18, 64)) > 0          # overlapping input tiler
+    P, F = [[1, 0, 0], [0, 8, 0], [0, 0, 8]], [[0, 0], [1, 0], [0, 1]]
+    for origin in ([0, 0, 0], [0, -3, 5]):                              # SURVEY d3 blocking, plain and wrapping
+        assert ws(aol.make_tiler([64, 1024, 1024], [64, 128, 128], [8, 8], origin, P, F)) == 0
+    assert ws(aol.make_tiler([7], [7], [], [3], [[-1]], [[]])) == 0     # reversal (coefficient -1)
+    assert ws(aol.make_tiler([8], [2], [5], [0], [[4]], [[1]])) == 8 * 4   # overlapping windows: claims
+
+
 def test_workspace_bytes():
     t = aol.make_tiler([4, 5], [2], [3], [0, 0], [[1], [2]], [[0], [1]])
-    assert _lib.lib().aol_tiler_scatter_workspace_bytes(ctypes.byref(t)) == 20 * 8
+    # the repetition dim moves both array dims: injectivity not provable -> 4-byte claims per element
+    assert _lib.lib().aol_tiler_scatter_workspace_bytes(ctypes.byref(t)) == 20 * 4
     assert _lib.lib().aol_tiler_scatter_workspace_bytes(None) == 0
     L = _lib.lib()
     assert L.aol_downscale_frame_host_workspace_bytes(_lib.I32, 4, 3, 1080, 1920) > 2 * 4 * 3 * 1080 * 1920 * 4

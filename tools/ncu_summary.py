@@ -1,9 +1,12 @@
 #!/usr/bin/env python
 """Summarise an `ncu --set full` capture and a launch list into profiles/.
 
-usage: python tools/ncu_summary.py <prof.ncu-rep> <launches.csv> <tag> <workload-key>
+usage: python tools/ncu_summary.py <prof.ncu-rep> <launches.csv|-> <tag> <workload-key> [<bench-log>]
 Writes profiles/<tag>_ncu_full.txt, profiles/<tag>_launches.csv and merges the per-launch
-DRAM bytes into profiles/ncu_traffic.json (read by bench.py for roofline.traffic).
+DRAM bytes into profiles/ncu_traffic.json (read by bench.py for roofline.traffic).  The entry is
+keyed by the source-tree hash and launch plan of the captured run, taken from the bench.py JSON
+line in <bench-log> (the stdout of the command ncu profiled), so bench.py quotes it only for the
+same tree and launch.
 """
 import csv
 import io
@@ -32,8 +35,17 @@ def raw(rep):
     return rows[0], rows[1], rows[2:]
 
 
+def bench_line(path):
+    with open(path) as f:
+        for line in f:
+            if line.startswith("{"):
+                return json.loads(line)
+    return None
+
+
 def main():
     rep, launches, tag, key = sys.argv[1:5]
+    bl = bench_line(sys.argv[5]) if len(sys.argv) > 5 else None
     hdr, units, rows = raw(rep)
     lines = [f"# ncu --set full summary: {os.path.basename(rep)} (tag {tag}, workload {key})"]
     per = []
@@ -55,7 +67,10 @@ def main():
         v = float(v.replace(",", ""))
         return v * {"byte": 1, "Kbyte": 1e3, "Mbyte": 1e6, "Gbyte": 1e9, "Tbyte": 1e12}.get(u, 1)
 
-    if per:
+    if per and bl is not None:
+        sys.path.insert(0, ROOT)
+        import bench
+
         d = per[-1]
         rb = to_bytes(*d["dram__bytes_read.sum"])
         wb = to_bytes(*d["dram__bytes_write.sum"])
@@ -63,9 +78,13 @@ def main():
         allv = json.load(open(path)) if os.path.exists(path) else {}
         allv[key] = {"dram_bytes_per_launch": rb + wb, "dram_read": rb, "dram_write": wb, "tag": tag,
                      "duration": d["gpu__time_duration.sum"][0] + " " + d["gpu__time_duration.sum"][1],
-                     "dram_pct_of_peak": float(d["gpu__dram_throughput.avg.pct_of_peak_sustained_elapsed"][0])}
+                     "dram_pct_of_peak": float(d["gpu__dram_throughput.avg.pct_of_peak_sustained_elapsed"][0]),
+                     "src_hash": bl["launch"]["src_hash"], "plan": bench.plan_key(bl["launch"]["plan"])}
         json.dump(allv, open(path, "w"), indent=1)
     # launch list
+    if launches == "-":
+        print("\n".join(lines[:40]))
+        return
     with open(launches) as f:
         txt = f.read()
     rows = [r for r in csv.reader(io.StringIO(txt[txt.index('"ID"'):]))]
