@@ -451,18 +451,60 @@ def record_d1(aol, peak, check):
                 call()
     torch.cuda.synchronize()
     graph_ms, _ = timed(lambda: g.replay(), reps=20)
+    # the same call through a persistent plan (aol_frame_plan_*): one kernel launch, no per-call planning
+    zp = torch.empty_like(z)
+    csp = torch.empty_like(cs)
+    plan = aol.FramePlan(x, out=zp, checksums=csp)
+    pwarm, _ = timed(plan.launch, reps=50, before=lambda: torch.cuda._sleep(200000))
+    torch.cuda.synchronize()
+    t0 = time.perf_counter()
+    for _ in range(200):
+        plan.launch()
+    plan_host_us = (time.perf_counter() - t0) / 200 * 1e6
+    torch.cuda.synchronize()
+    gp = torch.cuda.CUDAGraph()
+    sp = torch.cuda.Stream()
+    sp.wait_stream(torch.cuda.current_stream())
+    with torch.cuda.stream(sp):
+        plan_g = aol.FramePlan(x, out=zp, checksums=csp, stream=sp)
+        plan_g.launch()
+        torch.cuda.synchronize()
+        with torch.cuda.graph(gp, stream=sp):
+            for _ in range(20):
+                plan_g.launch()
+    torch.cuda.synchronize()
+    pgraph_ms, _ = timed(lambda: gp.replay(), reps=20)
+    torch.cuda.synchronize()
+    plan_ok = bool(torch.equal(zp, z) and torch.equal(csp.view(torch.int64), cs.view(torch.int64)))
+    # C-level host enqueue (examples/aol_example.c, no Python): plan launch vs aol_downscale_frame
+    c_enq = None
+    exe = os.path.join(ROOT, "build", "aol_example")
+    if os.path.exists(exe):
+        import subprocess
+
+        r = subprocess.run([exe, "--enqueue-us", "2000"], capture_output=True, text=True, timeout=120)
+        if r.returncode == 0 and r.stdout.strip():
+            c_enq = json.loads(r.stdout.strip().splitlines()[-1])
     b = frame_bytes(C, H, W)
     rec = {"config": "d1 single 1920x1080 3-channel frame -> 720x480 (BASELINE configs[0])",
            "warm_l2_us": warm * 1e3, "cold_l2_us": cold * 1e3, "graph_us_per_call": graph_ms * 1e3 / 20,
            "host_enqueue_us_per_call_python": host_us, "roofline_floor_us": b / peak / 1e3,
+           "plan": {"warm_l2_us": pwarm * 1e3, "graph_us_per_call": pgraph_ms * 1e3 / 20,
+                    "host_enqueue_us_per_call_python": plan_host_us,
+                    "host_enqueue_us_per_call_c": c_enq["plan_launch_us"] if c_enq else None,
+                    "same_outputs_as_downscale_frame": plan_ok,
+                    "note": "aol_frame_plan_launch: one kernel launch (checksum partials + self-resetting "
+                            "per-frame counters instead of the zeroing kernel)"},
+           "host_enqueue_us_per_call_c": c_enq["downscale_frame_us"] if c_enq else None,
            "frac_cold": (b / peak / 1e3) / (cold * 1e3), "frac_graph": (b / peak / 1e3) / (graph_ms * 1e3 / 20),
            "timing": "CUDA events, median of 50 (warm: 200 us GPU sleep before each call; cold: 512 MB fill before "
-                     "each call); graph: 20 calls per replay, median of 20",
-           "plan": aol.downscale_frame_plan(N, C, H, W)}
+                     "each call); graph: 20 calls per replay, median of 20; host enqueue: wall clock over 200 "
+                     "calls (python) / 2000 calls (C, examples/aol_example.c --enqueue-us)",
+           "launch_plan": aol.downscale_frame_plan(N, C, H, W)}
     torch.cuda.synchronize()
     rec["_parity_args"] = (seed, 0, C, H, W, z.cpu().numpy(), cs.cpu().view(torch.int64).numpy().view(np.uint64))
     if check:
-        rec["parity"] = cpu_parity_frame(*rec["_parity_args"])
+        rec["parity"] = cpu_parity_frame(*rec["_parity_args"]) and plan_ok
     del rec["_parity_args"]
     return rec
 

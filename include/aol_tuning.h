@@ -31,6 +31,11 @@ extern "C" {
  * check that a failing call enqueues nothing -- the caller's output and checksum buffers stay untouched. */
 AOL_API void aol_debug_fail_next_launches(int n);
 
+/* Name of the last kernel an aol_* call launched on this thread (e.g. "tiler_box_kernel",
+ * "fused_tma_kernel"); "" before any launch.  Lets tests and reports check which kernel path a
+ * descriptor or shape takes. */
+AOL_API const char* aol_debug_last_kernel(void);
+
 #ifdef __cplusplus
 }
 #endif

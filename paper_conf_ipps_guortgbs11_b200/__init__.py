@@ -26,7 +26,7 @@ from ._lib import (FILTER_H, FILTER_V, AolError, I16, I32, I64, PRESET_H_IN, PRE
 __all__ = [
     "AolError", "version", "make_tiler", "tiler_preset", "tiler_validate", "tiler_is_injective",
     "tiler_gather", "tiler_scatter", "tiler_scatter_workspace_bytes", "downscale_h", "downscale_v", "downscale_frame", "downscale_frame_plan",
-    "frame_checksum", "downscale_frame_host", "synth_frames", "library_path", "downscale_frame_packed",
+    "frame_checksum", "downscale_frame_host", "FramePlan", "synth_frames", "library_path", "downscale_frame_packed",
     "PRESET_H_IN", "PRESET_H_OUT", "PRESET_V_IN", "PRESET_V_OUT", "SYNTH_KINDS",
     "make_filter", "filter_preset", "filter_validate", "filter_apply", "FILTER_H", "FILTER_V", "FLAGS",
 ]
@@ -77,6 +77,11 @@ def _dev(t: torch.Tensor, name: str) -> ctypes.c_void_p:
 
 def version() -> int:
     return int(lib().aol_version())
+
+
+def last_kernel() -> str:
+    """Name of the last kernel a library call launched on this thread (aol_debug_last_kernel)."""
+    return lib().aol_debug_last_kernel().decode()
 
 
 # ------------------------------------------------------------------ tilers
@@ -306,6 +311,67 @@ def downscale_frame_packed(x: torch.Tensor, out: Optional[torch.Tensor] = None, 
         check(lib().aol_downscale_frame_out(_dev(x, "x"), RGB8, _dev(out, "out"), _TYPED[odt], N, 3, H, W, cs_ptr,
                                             ctypes.byref(o) if o is not None else None, _stream(stream, x.device)))
     return out, cs
+
+
+class FramePlan:
+    """A persistent launch plan (aol_frame_plan_*): the fused downscale of fixed tensors x -> out resolved once;
+    launch() is then one kernel launch (the d1 single-frame case).  x: planar int32/uint8 [N][C][H][W], or
+    packed uint8 [N][H][W][3] with packed=True.  Keep x / out / checksums alive while the plan is used;
+    launches of one plan must be stream-ordered."""
+
+    def __init__(self, x: torch.Tensor, out: Optional[torch.Tensor] = None, checksums=None, opts=None,
+                 out_dtype: Optional[torch.dtype] = None, packed: bool = False, stream=None):
+        if packed:
+            if x.dim() != 4 or x.shape[3] != 3 or x.dtype != torch.uint8:
+                raise ValueError("packed x must be uint8 [frames][H][W][3]")
+            N, H, W, C = x.shape
+            code = RGB8
+        else:
+            if x.dim() != 4 or x.dtype not in (torch.int32, torch.uint8):
+                raise ValueError("x must be int32 or uint8 [frames][channels][H][W]")
+            N, C, H, W = x.shape
+            code = _TYPED[x.dtype]
+        odt = out.dtype if out is not None else (out_dtype or torch.int32)
+        if out is None:
+            out = torch.empty((N, C, 4 * (H // 9), 3 * (W // 8)), dtype=odt, device=x.device)
+        _out(out, (N, C, 4 * (H // 9), 3 * (W // 8)), odt, x.device, "out")
+        if checksums is True:
+            checksums = torch.empty(N, dtype=torch.uint64, device=x.device)
+        self.x, self.out, self.checksums = x, out, checksums
+        self._cs = (_dev(_checksum_buf(checksums, N, x.device), "checksums") if checksums is not None
+                    else ctypes.c_void_p(0))
+        self._h = ctypes.c_void_p(0)
+        o = _opts(opts)
+        self._lib = lib()
+        with torch.cuda.device(x.device):
+            check(self._lib.aol_frame_plan_create(_dev(x, "x"), code, _dev(out, "out"), _TYPED[odt], N, C, H, W,
+                                                  ctypes.byref(o) if o is not None else None, ctypes.byref(self._h)))
+        self._stream = _stream(stream, x.device)
+        self._launch = self._lib.aol_frame_plan_launch
+
+    def launch(self):
+        """Enqueue one downscale on the plan's stream (the current stream at creation unless given)."""
+        st = self._launch(self._h, self._cs, self._stream)
+        if st:
+            check(st)
+        return self.out, self.checksums
+
+    def info(self) -> dict:
+        p = aol_plan_t()
+        check(self._lib.aol_frame_plan_info(self._h, ctypes.byref(p)))
+        return {f: getattr(p, f) for f, _ in aol_plan_t._fields_}
+
+    def close(self):
+        if self._h:
+            check(self._lib.aol_frame_plan_destroy(self._h))
+            self._h = ctypes.c_void_p(0)
+
+    def __del__(self):
+        try:
+            if self._h:
+                self._lib.aol_frame_plan_destroy(self._h)
+        except Exception:
+            pass
 
 
 def downscale_frame_plan(frames: int, channels: int, H: int, W: int, dtype=torch.int32, opts=None,

@@ -112,6 +112,12 @@ SIGNATURES = {
     "aol_filter_validate": ([_FP], _ST),
     "aol_filter_apply": ([_FP, _P, _P, _P], _ST),
     "aol_debug_fail_next_launches": ([ctypes.c_int], None),
+    "aol_debug_last_kernel": ([], ctypes.c_char_p),
+    "aol_frame_plan_create": ([_P, ctypes.c_int, _P, ctypes.c_int, _I64, _I64, _I64, _I64,
+                               ctypes.POINTER(aol_launch_opts_t), ctypes.POINTER(_P)], _ST),
+    "aol_frame_plan_launch": ([_P, _P, _P], _ST),
+    "aol_frame_plan_info": ([_P, ctypes.POINTER(aol_plan_t)], _ST),
+    "aol_frame_plan_destroy": ([_P], _ST),
     "aol_synth_frames": ([ctypes.c_uint64, _I64, _I64, _I64, _I64, _I64, _I32, _I32, ctypes.c_int, _P, _P], _ST),
 }
 

@@ -104,14 +104,23 @@ int kernel_occupancy(const void* fn, int block, int smem) {
 
 namespace {
 thread_local int g_fail_launches = 0;   // aol_debug_fail_next_launches (test hook)
+thread_local const char* g_last_kernel = "";
 }
 
-aol_status_t launch_preflight(const void* fn, int block, int smem, const char* what) {
+void note_launch(const char* what) { g_last_kernel = what; }
+
+aol_status_t debug_injected_failure(const char* what) {
     if (g_fail_launches > 0) {
         --g_fail_launches;
         set_error("launch of %s failed: injected failure (aol_debug_fail_next_launches)", what);
         return AOL_E_CUDA;
     }
+    return AOL_OK;
+}
+
+aol_status_t launch_preflight(const void* fn, int block, int smem, const char* what) {
+    aol_status_t st = debug_injected_failure(what);
+    if (st != AOL_OK) return st;
     if (kernel_occupancy(fn, block, smem) < 1) {
         set_error("launch of %s is not runnable: %d threads with %d bytes of dynamic shared memory", what, block,
                   smem);
@@ -348,14 +357,36 @@ aol_status_t check_opts(const aol_launch_opts_t* opts) {
     return AOL_OK;
 }
 
+}  // namespace
+
+aol_status_t aol::validate_frame_call(const void* d_in, aol_dtype_t in_dtype, const void* d_out,
+                                      aol_dtype_t out_dtype, int64_t frames, int64_t channels, int64_t H, int64_t W,
+                                      const uint64_t* d_cs, const aol_launch_opts_t* opts) {
+    aol_status_t st = check_frame_args(d_in, in_dtype, d_out, frames, channels, H, W, out_dtype, d_cs);
+    if (st != AOL_OK) return st;
+    return check_opts(opts);
+}
+
+void aol::fill_plan_info(const FusedPlan& p, aol_plan_t* out) {
+    out->kernel = p.kernel;
+    out->grid = p.grid;
+    out->block = p.block;
+    out->smem_bytes = p.smem;
+    out->stages = p.stages;
+    out->bands_per_unit = p.bands_per_unit;
+    out->units = p.units;
+    out->ctas_per_sm = p.ctas_per_sm;
+    out->num_sms = p.num_sms;
+}
+
+namespace {
+
 aol_status_t frame_ex(const void* d_in, aol_dtype_t in_dtype, void* d_out, aol_dtype_t out_dtype, int64_t frames,
                       int64_t channels, int64_t H, int64_t W, uint64_t* d_cs, const aol_launch_opts_t* opts,
                       cudaStream_t s) {
-    aol_status_t st = check_frame_args(d_in, in_dtype, d_out, frames, channels, H, W, out_dtype, d_cs);
+    aol_status_t st = validate_frame_call(d_in, in_dtype, d_out, out_dtype, frames, channels, H, W, d_cs, opts);
     if (st != AOL_OK) return st;
     if (frames == 0) return AOL_OK;
-    st = check_opts(opts);
-    if (st != AOL_OK) return st;
     FusedPlan plan;
     st = plan_fused(in_dtype, out_dtype, d_in, d_out, frames, channels, H, W, opts, &plan);
     if (st != AOL_OK) return st;
@@ -369,6 +400,8 @@ extern "C" {
 int aol_version(void) { return AOL_VERSION; }
 
 void aol_debug_fail_next_launches(int n) { g_fail_launches = n > 0 ? n : 0; }
+
+const char* aol_debug_last_kernel(void) { return g_last_kernel; }
 
 const char* aol_last_error(void) { return aol::last_error_cstr(); }
 
@@ -555,15 +588,7 @@ aol_status_t aol_downscale_frame_plan_out(aol_dtype_t in_dtype, aol_dtype_t out_
     FusedPlan p;
     st = plan_fused(in_dtype, out_dtype, nullptr, nullptr, frames, channels, H, W, opts, &p);
     if (st != AOL_OK) return st;
-    out->kernel = p.kernel;
-    out->grid = p.grid;
-    out->block = p.block;
-    out->smem_bytes = p.smem;
-    out->stages = p.stages;
-    out->bands_per_unit = p.bands_per_unit;
-    out->units = p.units;
-    out->ctas_per_sm = p.ctas_per_sm;
-    out->num_sms = p.num_sms;
+    fill_plan_info(p, out);
     return AOL_OK;
 }
 

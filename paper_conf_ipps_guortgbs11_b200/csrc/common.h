@@ -32,9 +32,13 @@ inline aol_status_t fail(aol_status_t st, const char* what) {
         }                                                                                             \
     } while (0)
 
+// Name of the last kernel this thread launched (aol_debug_last_kernel, a test / report hook).
+void note_launch(const char* what);
+
 // After a launch: report launch-configuration errors synchronously.
 #define AOL_LAUNCH_CHECK(what)                                                                        \
     do {                                                                                              \
+        ::aol::note_launch(what);                                                                     \
         cudaError_t err__ = cudaGetLastError();                                                       \
         if (err__ != cudaSuccess) {                                                                   \
             ::aol::set_error("launch of %s failed: %s", what, cudaGetErrorString(err__));             \
@@ -57,6 +61,7 @@ int kernel_occupancy(const void* fn, int block, int smem);  // resident CTAs per
 // and the test hook aol_debug_fail_next_launches() may force a failure here.  Called before the FIRST
 // enqueue of an entry point, so a failing call leaves the caller's buffers untouched.
 aol_status_t launch_preflight(const void* fn, int block, int smem, const char* what);
+aol_status_t debug_injected_failure(const char* what);   // the test hook alone (AOL_OK unless armed)
 
 // ---- launchers implemented in the .cu files (all validate nothing; callers do)
 struct FusedPlan {
@@ -66,6 +71,13 @@ struct FusedPlan {
     int out_es;           // output element bytes: 4 (int32) or 2 (int16, uint8 input only)
     int64_t units;
 };
+
+// Argument checks of the fused entry points (shapes, dtypes, alignment incl. the checksum pointer, options).
+aol_status_t validate_frame_call(const void* d_in, aol_dtype_t in_dtype, const void* d_out, aol_dtype_t out_dtype,
+                                 int64_t frames, int64_t channels, int64_t H, int64_t W, const uint64_t* d_cs,
+                                 const aol_launch_opts_t* opts);
+struct FusedPlan;
+void fill_plan_info(const FusedPlan& p, aol_plan_t* out);
 
 aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void* d_in, const void* d_out,
                         int64_t frames, int64_t channels, int64_t H, int64_t W, const aol_launch_opts_t* opts,

@@ -310,42 +310,35 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void*
     return AOL_OK;
 }
 
-aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t in_dtype, void* d_out,
-                          int64_t frames, int64_t channels, int64_t H, int64_t W, uint64_t* d_cs, cudaStream_t s) {
+aol_status_t prepare_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t in_dtype, void* d_out,
+                           int64_t frames, int64_t channels, int64_t H, int64_t W, FusedLaunch* L) {
     const bool rgb = in_dtype == AOL_RGB8;
     const int64_t planes = rgb ? frames : frames * channels;   // packed pixels: work units per frame
-    const int32_t Ho = int32_t(4 * (H / 9)), Wo = int32_t(3 * (W / 8));
-
-    if (plan.kernel == 2) {
-        if (in_dtype == AOL_U8 && plan.out_es == 2)
-            return launch_generic<uint8_t, int16_t>(plan, d_in, d_out, d_cs, frames, planes, H, W, Ho, Wo, channels, s);
-        if (in_dtype == AOL_U8)
-            return launch_generic<uint8_t, int32_t>(plan, d_in, d_out, d_cs, frames, planes, H, W, Ho, Wo, channels, s);
-        return launch_generic<int32_t, int32_t>(plan, d_in, d_out, d_cs, frames, planes, H, W, Ho, Wo, channels, s);
-    }
-
-    CUtensorMap map;
-    std::memset(&map, 0, sizeof map);
+    std::memset(&L->map, 0, sizeof L->map);
     const bool u8_tensor = in_dtype == AOL_U8 && W % 128 == 0 && W / 128 <= 256 && planes * H < (int64_t(1) << 31);
     const int layout = i32_layout(in_dtype, W, plan.flags);
     if (layout > 0 || u8_tensor) {
-        aol_status_t st = encode_row_map(&map, in_dtype, d_in, planes * H, W, plan.flags);
+        aol_status_t st = encode_row_map(&L->map, in_dtype, d_in, planes * H, W, plan.flags);
         if (st != AOL_OK) return st;
     }
-    FusedArgs a;
+    FusedArgs& a = L->args;
+    std::memset(&a, 0, sizeof a);
     a.u8_tensor = u8_tensor ? 1 : 0;
     a.rows_per_stage = rows_per_stage(in_dtype, W, plan.flags);
     a.Z = d_out;
-    a.cs = d_cs;
     a.X = d_in;
     // units from THIS call's frame count (a plan may be reused for a shorter batch, e.g. the last chunk of
     // the host-streamed path): never more units, or CTAs, than the batch has
     a.nunits = planes * plan.units_per_plane;
-    const int grid = int(std::min<int64_t>(plan.grid, a.nunits));
+    L->grid = int(std::min<int64_t>(plan.grid, a.nunits));
+    L->block = plan.block;
+    L->smem = plan.smem;
+    L->frames = frames;
+    L->flags = plan.flags;
     a.H = int32_t(H);
     a.W = int32_t(W);
-    a.Ho = Ho;
-    a.Wo = Wo;
+    a.Ho = int32_t(4 * (H / 9));
+    a.Wo = int32_t(3 * (W / 8));
     a.channels = rgb ? 1 : int32_t(channels);   // packed: the unit index is the frame index
     a.row_pitch = int32_t(rgb ? 3 * W : W);
     a.reps = int32_t(W / 8);
@@ -354,30 +347,38 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
     a.nbands = int32_t(H / 9);
     a.bands_per_unit = plan.bands_per_unit;
     a.units_per_plane = plan.units_per_plane;
+    a.units_per_frame = int32_t((rgb ? 1 : channels) * plan.units_per_plane);
     a.stages = plan.stages;
     const RingGeom geom = ring_geom(in_dtype, plan.out_es, W, plan.flags);
     a.stage_bytes = geom.stage_bytes;
     a.stage_stride = geom.stage_stride;
     a.out_bytes = geom.out_bytes;
     a.n_consumer = plan.block - 32;
+    a.cs_mode = 0;
+    for (int c = 0; c < 2; ++c) {
+        L->k[c] = pick(in_dtype, plan.out_es, c == 1, plan.reps_per_thread, W, plan.flags, plan.block,
+                       plan.ctas_per_sm);
+        aol_status_t st = kernel_smem(reinterpret_cast<const void*>(L->k[c]), plan.smem);
+        if (st != AOL_OK) return st;
+    }
+    return AOL_OK;
+}
 
-    KernelFn k = pick(in_dtype, plan.out_es, d_cs != nullptr, plan.reps_per_thread, W, plan.flags, plan.block,
-                      plan.ctas_per_sm);
-    aol_status_t st_attr = kernel_smem(reinterpret_cast<const void*>(k), plan.smem);
-    if (st_attr != AOL_OK) return st_attr;
-    // Everything that can fail before the kernels run has been resolved (plan, tensor map, smem attribute);
-    // the pre-flight checks the configuration is runnable.  Nothing has been enqueued yet.
-    st_attr = launch_preflight(reinterpret_cast<const void*>(k), plan.block, plan.smem, "fused_tma_kernel");
-    if (st_attr != AOL_OK) return st_attr;
-    // With checksums: zero them in a one-CTA kernel and launch the fused kernel as its programmatic
+aol_status_t enqueue_fused(const FusedLaunch& L, uint64_t* d_cs, cudaStream_t s) {
+    FusedArgs a = L.args;
+    a.cs = d_cs;
+    KernelFn k = L.k[d_cs ? 1 : 0];
+    // With checksums (cs_mode 0): zero them in a one-CTA kernel and launch the fused kernel as its programmatic
     // dependent, so the zeroing (and the launch gap after it) overlaps the fused kernel's start instead of
     // preceding it (single-frame latency).  Only the zero kernel can be the primary: it
     // is an ordinary launch, so everything earlier in the stream (e.g. the producer of X) has completed.
     // PDL invariant: the fused kernel issues its TMA loads and bulk stores without griddepcontrol.wait, so it
     // may only be a programmatic dependent of zero_checksums_kernel (which touches nothing but cs and waits
     // for its own predecessor); pdl therefore requires d_cs, and the zero kernel is launched right before it.
-    const bool pdl = d_cs && !(plan.flags & AOL_FLAG_NO_PDL);
-    if (d_cs) {
+    // cs_mode 1 (plans) needs no zeroing: one launch.
+    const bool zero = d_cs && a.cs_mode == 0;
+    const bool pdl = zero && !(L.flags & AOL_FLAG_NO_PDL);
+    if (zero) {
         cudaLaunchConfig_t zc;
         std::memset(&zc, 0, sizeof zc);
         zc.gridDim = dim3(1);
@@ -388,31 +389,52 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
         za[0].val.programmaticStreamSerializationAllowed = 1;
         zc.attrs = za;
         zc.numAttrs = pdl ? 1 : 0;
-        cudaError_t ze = cudaLaunchKernelEx(&zc, zero_checksums_kernel, d_cs, int64_t(frames));
+        cudaError_t ze = cudaLaunchKernelEx(&zc, zero_checksums_kernel, d_cs, int64_t(L.frames));
         if (ze != cudaSuccess) {
             set_error("launch of zero_checksums_kernel failed: %s", cudaGetErrorString(ze));
             return AOL_E_CUDA;
         }
-        AOL_LAUNCH_CHECK("zero_checksums_kernel");
     }
     cudaLaunchConfig_t cfg;
     std::memset(&cfg, 0, sizeof cfg);
-    cfg.gridDim = dim3(unsigned(grid));
-    cfg.blockDim = dim3(unsigned(plan.block));
-    cfg.dynamicSmemBytes = size_t(plan.smem);
+    cfg.gridDim = dim3(unsigned(L.grid));
+    cfg.blockDim = dim3(unsigned(L.block));
+    cfg.dynamicSmemBytes = size_t(L.smem);
     cfg.stream = s;
     cudaLaunchAttribute attr[1];
     attr[0].id = cudaLaunchAttributeProgrammaticStreamSerialization;
     attr[0].val.programmaticStreamSerializationAllowed = 1;
     cfg.attrs = attr;
     cfg.numAttrs = pdl ? 1 : 0;
-    cudaError_t le = cudaLaunchKernelEx(&cfg, k, map, a);
+    cudaError_t le = cudaLaunchKernelEx(&cfg, k, L.map, a);
+    note_launch("fused_tma_kernel");
     if (le != cudaSuccess) {
         set_error("launch of fused_tma_kernel failed: %s", cudaGetErrorString(le));
         return AOL_E_CUDA;
     }
-    AOL_LAUNCH_CHECK("fused_tma_kernel");
     return AOL_OK;
+}
+
+aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t in_dtype, void* d_out,
+                          int64_t frames, int64_t channels, int64_t H, int64_t W, uint64_t* d_cs, cudaStream_t s) {
+    if (plan.kernel == 2) {
+        const bool rgb = in_dtype == AOL_RGB8;
+        const int64_t planes = rgb ? frames : frames * channels;
+        const int32_t Ho = int32_t(4 * (H / 9)), Wo = int32_t(3 * (W / 8));
+        if (in_dtype == AOL_U8 && plan.out_es == 2)
+            return launch_generic<uint8_t, int16_t>(plan, d_in, d_out, d_cs, frames, planes, H, W, Ho, Wo, channels, s);
+        if (in_dtype == AOL_U8)
+            return launch_generic<uint8_t, int32_t>(plan, d_in, d_out, d_cs, frames, planes, H, W, Ho, Wo, channels, s);
+        return launch_generic<int32_t, int32_t>(plan, d_in, d_out, d_cs, frames, planes, H, W, Ho, Wo, channels, s);
+    }
+    FusedLaunch L;
+    aol_status_t st = prepare_fused(plan, d_in, in_dtype, d_out, frames, channels, H, W, &L);
+    if (st != AOL_OK) return st;
+    // Everything that can fail before the kernels run has been resolved (plan, tensor map, smem attributes);
+    // the pre-flight checks the configuration is runnable.  Nothing has been enqueued yet.
+    st = launch_preflight(reinterpret_cast<const void*>(L.k[d_cs ? 1 : 0]), L.block, L.smem, "fused_tma_kernel");
+    if (st != AOL_OK) return st;
+    return enqueue_fused(L, d_cs, s);
 }
 
 }  // namespace aol

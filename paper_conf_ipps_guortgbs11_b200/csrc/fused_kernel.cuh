@@ -45,6 +45,7 @@
 #include <cstdint>
 #include <type_traits>
 
+#include "common.h"
 #include "ptx.cuh"
 
 namespace aol {
@@ -116,6 +117,14 @@ struct FusedArgs {
     int32_t rows_per_stage; // int32 path: 3 (a stage holds a row triple) or 1 (one row per stage: finer ring
                             // granularity for wide frames); always 3 for uint8
     int32_t row_pitch;      // uint8 paths: bytes per input row (W planar, 3W packed 24-bit pixels)
+    // Checksum epilogue.  cs_mode 0: one atomicAdd per unit into cs, which zero_checksums_kernel cleared first.
+    // cs_mode 1 (plan launches, aol_frame_plan_launch): no zeroing kernel -- each unit stores its partial sum in
+    // cs_partial[unit] and counts itself in cs_count[frame]; the frame's last unit sums the partials into
+    // cs[frame] and resets the counter to 0 for the next launch (self-resetting, one launch per call).
+    int32_t cs_mode;
+    int32_t units_per_frame;    // cs_mode 1: work units of one frame (contiguous unit indices)
+    unsigned long long* cs_partial;
+    unsigned int* cs_count;
 };
 
 // Byte offset of 16-byte chunk `chunk` (0..7) of 128-byte line `line` under SWIZZLE_128B
@@ -587,11 +596,26 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
             if (tid == 0) {
                 unsigned long long sum = 0;
                 for (int w = 0; w < NC / 32; ++w) sum += red[w];
-                // the checksums were zeroed by the preceding zero_checksums_kernel, which this launch may
-                // overlap (programmatic dependent launch): wait for it before the first atomic (no-op when
-                // the kernel was launched without the PDL attribute, and after the first wait)
-                ptx::griddep_wait();
-                atomicAdd(reinterpret_cast<unsigned long long*>(a.cs + plane / a.channels), sum);
+                const int64_t frame = plane / a.channels;
+                if (a.cs_mode == 0) {
+                    // the checksums were zeroed by the preceding zero_checksums_kernel, which this launch may
+                    // overlap (programmatic dependent launch): wait for it before the first atomic (no-op when
+                    // the kernel was launched without the PDL attribute, and after the first wait)
+                    ptx::griddep_wait();
+                    atomicAdd(reinterpret_cast<unsigned long long*>(a.cs + frame), sum);
+                } else {
+                    a.cs_partial[u] = sum;
+                    __threadfence();   // the partial is visible before the count that publishes it
+                    const unsigned prev = atomicAdd(a.cs_count + frame, 1u);
+                    if (prev == unsigned(a.units_per_frame - 1)) {   // the frame's last unit
+                        __threadfence();
+                        const int64_t u0 = frame * a.units_per_frame;
+                        unsigned long long tot = 0;
+                        for (int32_t j = 0; j < a.units_per_frame; ++j) tot += __ldcg(a.cs_partial + u0 + j);
+                        a.cs[frame] = tot;
+                        a.cs_count[frame] = 0u;   // ready for the next launch (stream-ordered after this grid)
+                    }
+                }
             }
             ptx::named_bar_sync(2, NC);   // red[] is reused by the next unit
         }
@@ -676,10 +700,30 @@ __global__ void __launch_bounds__(256)
 
 using KernelFn = void (*)(const CUtensorMap, const FusedArgs);
 
+// A resolved fused-kernel launch (kernel 1): tensor map, arguments, the kernels without / with the checksum
+// epilogue (k[0] / k[1], smem attributes set), launch shape.  Built by prepare_fused (fused.cu), enqueued by
+// enqueue_fused: zero_checksums_kernel + the PDL fused launch for cs_mode 0, one launch for cs_mode 1.
+// Plans (plan.cu) keep one and re-enqueue it.
+struct FusedLaunch {
+    CUtensorMap map;
+    FusedArgs args;
+    KernelFn k[2];
+    int grid, block, smem, flags;
+    int64_t frames;
+};
+
 // Explicit instantiations live in fused_k_*.cu (compiled in parallel); these pick one.
 KernelFn tma_kernel_i32(bool checksum, int layout, int block, int cps);   // layout = kSwz (128 or 0)
 KernelFn tma_kernel_u8(bool checksum, bool out16, int reps_per_thread, int block, int cps);
 KernelFn tma_kernel_rgb8(bool checksum, bool out16, int block, int cps);   // packed 24-bit pixels
+
+}  // namespace fused
+
+aol_status_t prepare_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t in_dtype, void* d_out,
+                           int64_t frames, int64_t channels, int64_t H, int64_t W, fused::FusedLaunch* L);
+aol_status_t enqueue_fused(const fused::FusedLaunch& L, uint64_t* d_cs, cudaStream_t s);
+
+namespace fused {
 
 template <typename Tin, typename Tout, int kR, int kSwz, bool kChecksum>
 KernelFn pick_tma_kernel(int block, int cps) {

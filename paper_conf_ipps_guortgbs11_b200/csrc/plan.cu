@@ -1,0 +1,118 @@
+// plan.cu -- persistent launch plans for the fused downscaler (aol_frame_plan_*, include/aol.h).
+//
+// aol_downscale_frame re-plans every call: argument checks, the unit-size search, the TMA descriptor
+// encode, kernel-attribute lookups and two launches (checksum zeroing + the PDL fused kernel).  For one HD
+// frame that host work is longer than the kernel (the paper's own launch-overhead argument,
+// P:L776-779).  A plan resolves all of it once for fixed buffers and shape; a launch is then ONE
+// cudaLaunchKernelEx: the fused kernel's checksum epilogue runs in cs_mode 1 (per-unit partial sums and a
+// self-resetting per-frame counter in the plan's small device workspace), so no zeroing kernel is needed.
+#include <cuda_runtime.h>
+
+#include <cstring>
+#include <new>
+
+#include "common.h"
+#include "fused_kernel.cuh"
+
+struct aol_frame_plan {
+    aol::FusedPlan plan;
+    aol::fused::FusedLaunch launch;   // kernel 1
+    const void* d_in;
+    void* d_out;
+    aol_dtype_t in_dtype;
+    int64_t frames, channels, H, W;
+    void* d_ws;   // cs_mode 1: [units] u64 partial sums, then [frames] u32 counters (zero between launches)
+    int device;
+};
+
+using namespace aol;
+
+extern "C" {
+
+aol_status_t aol_frame_plan_create(const void* d_in, aol_dtype_t in_dtype, void* d_out, aol_dtype_t out_dtype,
+                                   int64_t frames, int64_t channels, int64_t H, int64_t W,
+                                   const aol_launch_opts_t* opts, aol_frame_plan_t* out) {
+    if (!out) return fail(AOL_E_INVALID, "out is NULL");
+    *out = nullptr;
+    if (frames <= 0) return fail(AOL_E_INVALID, "a plan needs frames > 0");
+    aol_status_t st = validate_frame_call(d_in, in_dtype, d_out, out_dtype, frames, channels, H, W, nullptr, opts);
+    if (st != AOL_OK) return st;
+    aol_frame_plan* p = new (std::nothrow) aol_frame_plan();
+    if (!p) return fail(AOL_E_INVALID, "out of host memory");
+    p->d_in = d_in;
+    p->d_out = d_out;
+    p->in_dtype = in_dtype;
+    p->frames = frames;
+    p->channels = channels;
+    p->H = H;
+    p->W = W;
+    p->d_ws = nullptr;
+    cudaGetDevice(&p->device);
+    st = plan_fused(in_dtype, out_dtype, d_in, d_out, frames, channels, H, W, opts, &p->plan);
+    if (st == AOL_OK && p->plan.kernel == 1) {
+        st = prepare_fused(p->plan, d_in, in_dtype, d_out, frames, channels, H, W, &p->launch);
+        for (int c = 0; c < 2 && st == AOL_OK; ++c)
+            st = launch_preflight(reinterpret_cast<const void*>(p->launch.k[c]), p->launch.block, p->launch.smem,
+                                  "fused_tma_kernel");
+        if (st == AOL_OK) {
+            const size_t units = size_t(p->launch.args.nunits);
+            const size_t bytes = units * 8 + size_t(frames) * 4;
+            cudaError_t e = cudaMalloc(&p->d_ws, bytes);
+            if (e == cudaSuccess) e = cudaMemset(static_cast<uint8_t*>(p->d_ws) + units * 8, 0, size_t(frames) * 4);
+            if (e == cudaSuccess) e = cudaDeviceSynchronize();   // counters are zero before any launch
+            if (e != cudaSuccess) {
+                set_error("plan workspace allocation failed: %s", cudaGetErrorString(e));
+                st = AOL_E_CUDA;
+            } else {
+                p->launch.args.cs_mode = 1;
+                p->launch.args.cs_partial = static_cast<unsigned long long*>(p->d_ws);
+                p->launch.args.cs_count = reinterpret_cast<unsigned int*>(static_cast<uint8_t*>(p->d_ws) + units * 8);
+            }
+        }
+    }
+    if (st != AOL_OK) {
+        if (p->d_ws) cudaFree(p->d_ws);
+        delete p;
+        return st;
+    }
+    *out = p;
+    return AOL_OK;
+}
+
+aol_status_t aol_frame_plan_launch(aol_frame_plan_t p, uint64_t* d_frame_checksums, cudaStream_t s) {
+    if (!p) return fail(AOL_E_INVALID, "plan is NULL");
+    if (reinterpret_cast<uintptr_t>(d_frame_checksums) % 8)
+        return fail(AOL_E_ALIGN, "d_frame_checksums must be 8-byte aligned");
+    if (p->plan.kernel != 1)   // the generic kernel: the ordinary two-step launch
+        return launch_fused(p->plan, p->d_in, p->in_dtype, p->d_out, p->frames, p->channels, p->H, p->W,
+                            d_frame_checksums, s);
+    aol_status_t st = debug_injected_failure("fused_tma_kernel");
+    if (st != AOL_OK) return st;
+    return enqueue_fused(p->launch, d_frame_checksums, s);
+}
+
+aol_status_t aol_frame_plan_info(aol_frame_plan_t p, aol_plan_t* out) {
+    if (!p || !out) return fail(AOL_E_INVALID, "NULL argument");
+    fill_plan_info(p->plan, out);
+    return AOL_OK;
+}
+
+aol_status_t aol_frame_plan_destroy(aol_frame_plan_t p) {
+    if (!p) return AOL_OK;
+    aol_status_t st = AOL_OK;
+    if (p->d_ws) {
+        int cur = 0;
+        cudaGetDevice(&cur);
+        cudaSetDevice(p->device);
+        cudaError_t e = cudaFree(p->d_ws);   // synchronising: pending launches of the plan finish first
+        cudaSetDevice(cur);
+        if (e != cudaSuccess) {
+            set_error("cudaFree of the plan workspace failed: %s", cudaGetErrorString(e));
+            st = AOL_E_CUDA;
+        }
+    }
+    delete p;
+    return st;
+}
+
+}  // extern "C"

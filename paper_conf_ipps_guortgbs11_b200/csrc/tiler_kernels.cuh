@@ -548,6 +548,369 @@ WrapTabDev make_wraptab(const Wrap32Dev& wd) {
     return wt;
 }
 
+// ------------------------------------------------------------ footprint-staged (box) tilers
+// Gathers / FAST scatters of tilers that wrap (the paper's H/V input tilers, Fig. 10; d3's wrapping
+// blockings) staged through shared memory.  The tile index space (natural order) splits into OUTER dims and
+// INNER dims (the innermost ones, the outermost of them possibly in chunks); for a fixed outer index the inner
+// block is CONTIGUOUS on the tile side and its array-side footprint lies in a BOX of raw coordinates
+//   [base_a, base_a + E_a)   per array dim a,   E_a = 1 + sum over inner dims |c_ad| (len_d - 1),
+// which wraps toroidally only when the box is loaded or stored (element (b_a) <-> array ((base_a + b_a) mod s_a)).
+// A CTA per block: (gather) load the box with coalesced row reads, the modulo applied once per row and per
+// row wrap point, into smem; then write the tile block with 16-byte vector stores, each element's smem offset
+// an affine function of its inner index (no modulo).  FAST scatter runs the same in reverse (tile block read
+// with vector loads, box written out row by row) when the inner block covers its box exactly (injective
+// tilers, ArrayOL single assignment).  Replaces the per-element offset arithmetic of the kernels above with
+// ~10 instructions per element and keeps both global sides streaming.
+constexpr int kBoxMaxInner = 4;           // inner dims (incl. the chunked one)
+constexpr int kBoxBytes = 48 * 1024;      // smem box per CTA (4 CTAs per SM)
+
+// Array dims are stored REVERSED in the box descriptors (r = 0 is the innermost, contiguous array dim: the box
+// row), so that every per-dim array is indexed by compile-time constants after unrolling (registers, no local
+// memory).
+struct BoxDev {
+    int32_t ra;                                            // array rank
+    int32_t ashape[AOL_MAX_RANK], astride[AOL_MAX_RANK];   // reversed
+    int32_t org[AOL_MAX_RANK];                             // origin (reduced mod s), reversed
+    // outer dims (enumerating blocks; the last one is the chunk index of the chunked inner dim)
+    int32_t n_out;
+    int32_t out_ext[2 * AOL_MAX_RANK + 1], out_g[2 * AOL_MAX_RANK + 1];
+    uint32_t out_mul[2 * AOL_MAX_RANK + 1], out_shift[2 * AOL_MAX_RANK + 1];
+    int32_t out_c[2 * AOL_MAX_RANK + 1][AOL_MAX_RANK];      // raw-coordinate step per outer dim (reversed)
+    // inner dims, outermost first: inner dim 0 is the chunked dim (length chunk_len, last chunk shorter)
+    int32_t n_in;
+    int32_t in_len[kBoxMaxInner];                          // full lengths (dim 0: chunk_len)
+    int32_t in_c[kBoxMaxInner][AOL_MAX_RANK];              // signed raw-coordinate step per inner dim (reversed)
+    int32_t chunk_ext, chunk_len;                          // extent of the chunked dim, chunk length
+    int32_t tail_prod;                                     // product of inner lengths after dim 0
+    uint32_t tail_mul, tail_shift;                         // magic division by tail_prod
+    uint32_t in_mul[kBoxMaxInner], in_shift[kBoxMaxInner]; // magic division by in_len (dims >= 1)
+    int32_t nblocks;
+    int32_t pitch_pad;                                     // extra elements per smem box row
+};
+
+__device__ __forceinline__ uint32_t magic_div(uint32_t n, uint32_t mul, uint32_t shift) {
+    return (__umulhi(n, mul) + n) >> shift;
+}
+
+// Per-block geometry: box extents / base coordinates (reversed dims) and the smem strides of the inner dims.
+struct BoxBlock {
+    int32_t g0, count;                 // tile-side start, elements in the block
+    int32_t len0;                      // this block's length of inner dim 0
+    int32_t E[AOL_MAX_RANK];           // box extents (E[0]: the row length)
+    int32_t base[AOL_MAX_RANK];        // box origin, reduced into [0, s)
+    int32_t step[kBoxMaxInner];        // smem offset per unit of inner dim d
+    int32_t off0;                      // smem offset of inner index 0
+    int32_t rows, pitch;
+};
+
+__device__ __forceinline__ void box_block(const BoxDev& bd, int32_t blk, BoxBlock& b) {
+    uint32_t n = uint32_t(blk);
+    int64_t raw[AOL_MAX_RANK];   // raw coordinates of the outer index (64-bit: sums of coef x index)
+#pragma unroll
+    for (int r = 0; r < AOL_MAX_RANK; ++r) raw[r] = r < bd.ra ? bd.org[r] : 0;
+    b.g0 = 0;
+    int32_t ck = 0;
+    for (int d = bd.n_out - 1; d >= 0; --d) {
+        const uint32_t q = magic_div(n, bd.out_mul[d], bd.out_shift[d]);
+        const int32_t i = int32_t(n - q * uint32_t(bd.out_ext[d]));
+        n = q;
+        if (d == bd.n_out - 1) ck = i;
+        b.g0 += bd.out_g[d] * i;
+#pragma unroll
+        for (int r = 0; r < AOL_MAX_RANK; ++r)
+            if (r < bd.ra) raw[r] += int64_t(bd.out_c[d][r]) * i;
+    }
+    b.len0 = min(bd.chunk_len, bd.chunk_ext - ck * bd.chunk_len);
+    b.count = b.len0 * bd.tail_prod;
+    // box extents, the corner's raw offset (negative steps reach below the outer index's raw point) and smem
+    // strides (r = 0: stride 1 along a row of pitch E[0] + pad; r > 0: products)
+    int32_t st = 1;
+    b.rows = 1;
+    b.off0 = 0;
+    int32_t bstride[AOL_MAX_RANK];
+#pragma unroll
+    for (int r = 0; r < AOL_MAX_RANK; ++r) {
+        b.E[r] = 1;
+        b.base[r] = 0;
+        bstride[r] = 0;
+        if (r >= bd.ra) continue;
+        int32_t lo = 0, hi = 0;
+#pragma unroll
+        for (int d = 0; d < kBoxMaxInner; ++d) {
+            if (d >= bd.n_in) continue;
+            const int32_t c = bd.in_c[d][r], l = (d == 0 ? b.len0 : bd.in_len[d]) - 1;
+            if (c < 0) lo += c * l; else hi += c * l;
+        }
+        b.E[r] = hi - lo + 1;
+        const int32_t v = int32_t((raw[r] + lo) % bd.ashape[r]);
+        b.base[r] = v < 0 ? v + bd.ashape[r] : v;
+        bstride[r] = st;
+        if (r == 0) {
+            b.pitch = b.E[0] + bd.pitch_pad;
+            st = b.pitch;
+        } else {
+            st *= b.E[r];
+            b.rows *= b.E[r];
+        }
+        b.off0 += -lo * bstride[r];   // smem offset of inner index 0
+    }
+#pragma unroll
+    for (int d = 0; d < kBoxMaxInner; ++d) {
+        int32_t o = 0;
+#pragma unroll
+        for (int r = 0; r < AOL_MAX_RANK; ++r)
+            if (r < bd.ra && d < bd.n_in) o += bd.in_c[d][r] * bstride[r];
+        b.step[d] = o;
+    }
+}
+
+// Global element offset of box row `row` (box dims r >= 1; r = 1 varies fastest).
+__device__ __forceinline__ int32_t box_row_offset(const BoxDev& bd, const BoxBlock& b, int32_t row) {
+    int32_t off = 0;
+#pragma unroll
+    for (int r = 1; r < AOL_MAX_RANK; ++r) {
+        if (r >= bd.ra) continue;
+        const int32_t q = row / b.E[r];
+        int32_t v = b.base[r] + (row - q * b.E[r]);
+        row = q;
+        while (v >= bd.ashape[r]) v -= bd.ashape[r];
+        off += v * bd.astride[r];
+    }
+    return off;
+}
+
+// Smem offset of the box element holding inner element e of the block (e < count).
+__device__ __forceinline__ int32_t box_inner_offset(const BoxDev& bd, const BoxBlock& b, uint32_t e,
+                                                    int32_t (&idx)[kBoxMaxInner]) {
+    const uint32_t i0 = magic_div(e, bd.tail_mul, bd.tail_shift);
+    uint32_t rem = e - i0 * uint32_t(bd.tail_prod);
+    idx[0] = int32_t(i0);
+    int32_t off = b.off0 + b.step[0] * int32_t(i0);
+#pragma unroll
+    for (int d = kBoxMaxInner - 1; d >= 1; --d) {
+        if (d >= bd.n_in) continue;
+        const uint32_t q = magic_div(rem, bd.in_mul[d], bd.in_shift[d]);
+        const int32_t i = int32_t(rem - q * uint32_t(bd.in_len[d]));
+        rem = q;
+        idx[d] = i;
+        off += b.step[d] * i;
+    }
+    return off;
+}
+
+// Advance the inner index by one (odometer over the inner dims, innermost last).
+__device__ __forceinline__ void box_inner_next(const BoxDev& bd, const BoxBlock& b, int32_t (&idx)[kBoxMaxInner],
+                                               int32_t& off) {
+#pragma unroll
+    for (int d = kBoxMaxInner - 1; d >= 0; --d) {
+        if (d >= bd.n_in) continue;
+        const int32_t len = d == 0 ? b.len0 : bd.in_len[d];
+        off += b.step[d];
+        if (++idx[d] < len) return;
+        idx[d] = 0;
+        off -= b.step[d] * len;
+    }
+}
+
+template <int ES, int VW, int MODE>
+__global__ void __launch_bounds__(256) tiler_box_kernel(const __grid_constant__ BoxDev bd, const void* __restrict__ src,
+                                                        void* __restrict__ dst) {
+    using T = typename Elem<ES>::T;
+    using VT = typename Vec<ES * VW>::T;
+    extern __shared__ __align__(16) uint8_t box_raw[];
+    T* box = reinterpret_cast<T*>(box_raw);
+    const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+    const int sl = bd.ashape[0];
+    for (int32_t blk = blockIdx.x; blk < bd.nblocks; blk += gridDim.x) {
+        BoxBlock b;
+        box_block(bd, blk, b);
+        const int32_t El = b.E[0], c0 = b.base[0];
+        if (MODE == 0) {
+            // ---- load the box: a warp per row, lanes along the row (coalesced), wrap at the row's end
+            const T* A = static_cast<const T*>(src);
+            for (int32_t row = warp; row < b.rows; row += 8) {
+                const int32_t roff = box_row_offset(bd, b, row);
+                T* srow = box + row * b.pitch;
+                constexpr int kU = 4;
+                for (int32_t x0 = lane; x0 < El; x0 += 32 * kU) {
+                    T v[kU];
+#pragma unroll
+                    for (int u = 0; u < kU; ++u) {
+                        const int32_t x = x0 + 32 * u;
+                        int32_t gc = c0 + x;
+                        while (gc >= sl) gc -= sl;
+                        if (x < El) v[u] = A[roff + gc];
+                    }
+#pragma unroll
+                    for (int u = 0; u < kU; ++u)
+                        if (x0 + 32 * u < El) srow[x0 + 32 * u] = v[u];
+                }
+            }
+            __syncthreads();
+            // ---- write the tile block: VW consecutive tile elements per thread (16-byte stores)
+            T* Tg = static_cast<T*>(dst) + b.g0;
+            for (int32_t v = threadIdx.x; v * VW < b.count; v += 256) {
+                int32_t idx[kBoxMaxInner] = {0, 0, 0, 0};
+                int32_t off = box_inner_offset(bd, b, uint32_t(v * VW), idx);
+                union { VT vec; T e[VW]; } pk;
+#pragma unroll
+                for (int j = 0; j < VW; ++j) {
+                    pk.e[j] = box[off];
+                    if (j + 1 < VW) box_inner_next(bd, b, idx, off);
+                }
+                reinterpret_cast<VT*>(Tg)[v] = pk.vec;
+            }
+            __syncthreads();   // the box is reloaded by the next block
+        } else {
+            // ---- FAST scatter: the tile block into the box (it covers the box exactly), then the box out
+            const T* Tg = static_cast<const T*>(src) + b.g0;
+            for (int32_t v = threadIdx.x; v * VW < b.count; v += 256) {
+                union { VT vec; T e[VW]; } pk;
+                pk.vec = reinterpret_cast<const VT*>(Tg)[v];
+                int32_t idx[kBoxMaxInner] = {0, 0, 0, 0};
+                int32_t off = box_inner_offset(bd, b, uint32_t(v * VW), idx);
+#pragma unroll
+                for (int j = 0; j < VW; ++j) {
+                    box[off] = pk.e[j];
+                    if (j + 1 < VW) box_inner_next(bd, b, idx, off);
+                }
+            }
+            __syncthreads();
+            T* A = static_cast<T*>(dst);
+            for (int32_t row = warp; row < b.rows; row += 8) {
+                const int32_t roff = box_row_offset(bd, b, row);
+                const T* srow = box + row * b.pitch;
+                for (int32_t x = lane; x < El; x += 32) {
+                    int32_t gc = c0 + x;
+                    while (gc >= sl) gc -= sl;
+                    A[roff + gc] = srow[x];
+                }
+            }
+            __syncthreads();
+        }
+    }
+}
+
+// Plan the box form of a tiler (fast32, every offset < 2^31); false if it does not qualify: the inner block
+// must be dense in its box (gather: box <= 1.5 x inner elements; scatter: exactly equal), box rows >= 32
+// elements long, <= kBoxMaxInner inner dims, box within kBoxBytes.
+bool make_box(const TilerDev& td, int es, int mode, BoxDev* bd, int* smem_bytes) {
+    if (!td.fast32 || td.array_elems >= (int64_t(1) << 31) || td.nd == 0) return false;
+    std::memset(bd, 0, sizeof *bd);
+    const int nd = td.nd, ra = td.ra;
+    int64_t sc[2 * AOL_MAX_RANK][AOL_MAX_RANK];   // signed raw steps (representative nearest 0)
+    for (int d = 0; d < nd; ++d)
+        for (int a = 0; a < ra; ++a) {
+            int64_t c = td.coef[a][d];
+            if (2 * c > td.ashape[a]) c -= td.ashape[a];
+            sc[d][a] = c;
+        }
+    auto box_of = [&](int k, int64_t lenk, int64_t* E) {   // inner = (chunk of dim k of length lenk), k+1..nd-1
+        int64_t vol = 1;
+        for (int a = 0; a < ra; ++a) {
+            int64_t span = 0;
+            for (int d = k; d < nd; ++d) {
+                const int64_t l = (d == k ? lenk : td.ext[d]) - 1;
+                span += (sc[d][a] < 0 ? -sc[d][a] : sc[d][a]) * l;
+            }
+            E[a] = span + 1;
+            vol *= E[a];
+            if (vol > (int64_t(1) << 40)) vol = int64_t(1) << 40;
+        }
+        return vol;
+    };
+    const int64_t budget = kBoxBytes / es;
+    // grow the inner block from the innermost dim outwards while the box fits; the first dim that does not fit
+    // entirely is chunked
+    int k = nd - 1;
+    int64_t E[AOL_MAX_RANK], lenk = td.ext[k];
+    for (;;) {
+        const int64_t pitch_extra = 4;
+        int64_t vol = box_of(k, td.ext[k], E);
+        if (vol + pitch_extra * (vol / std::max<int64_t>(1, E[ra - 1])) <= budget) {   // all of dim k fits
+            lenk = td.ext[k];
+            if (k == 0 || nd - (k - 1) > kBoxMaxInner) break;
+            int64_t E2[AOL_MAX_RANK];
+            const int64_t v2 = box_of(k - 1, 1, E2);   // would one slice of dim k-1 still fit?
+            if (v2 + pitch_extra * (v2 / std::max<int64_t>(1, E2[ra - 1])) > budget) break;
+            --k;
+            continue;
+        }
+        // chunk dim k: the largest length that fits
+        int64_t lo = 1, hi = td.ext[k];
+        while (lo < hi) {
+            const int64_t mid = (lo + hi + 1) / 2;
+            const int64_t v = box_of(k, mid, E);
+            if (v + pitch_extra * (v / std::max<int64_t>(1, E[ra - 1])) <= budget) lo = mid; else hi = mid - 1;
+        }
+        lenk = lo;
+        const int64_t v = box_of(k, lenk, E);
+        if (v + pitch_extra * (v / std::max<int64_t>(1, E[ra - 1])) > budget) return false;
+        break;
+    }
+    if (nd - k > kBoxMaxInner) return false;
+    const int64_t vol = box_of(k, lenk, E);
+    int64_t inner = lenk;
+    for (int d = k + 1; d < nd; ++d) inner *= td.ext[d];
+    if (mode == 0 ? (2 * vol > 3 * inner) : (vol != inner)) return false;
+    if (E[ra - 1] < 32) return false;
+    if (E[ra - 1] > 2 * td.ashape[ra - 1]) return false;   // the row wrap takes at most two subtractions
+    bd->ra = ra;
+    for (int a = 0; a < ra; ++a) {   // reversed: r = ra - 1 - a
+        bd->ashape[ra - 1 - a] = int32_t(td.ashape[a]);
+        bd->astride[ra - 1 - a] = int32_t(td.astride[a]);
+        bd->org[ra - 1 - a] = int32_t(td.org[a]);
+    }
+    int64_t gst[2 * AOL_MAX_RANK];
+    int64_t g = 1;
+    for (int d = nd - 1; d >= 0; --d) {
+        gst[d] = g;
+        g *= td.ext[d];
+    }
+    int no = 0;
+    for (int d = 0; d < k; ++d, ++no) {
+        bd->out_ext[no] = int32_t(td.ext[d]);
+        bd->out_g[no] = int32_t(gst[d]);
+        magic32(td.ext[d], &bd->out_mul[no], &bd->out_shift[no]);
+        for (int a = 0; a < ra; ++a) bd->out_c[no][ra - 1 - a] = int32_t(td.coef[a][d]);
+    }
+    const int64_t nch = (td.ext[k] + lenk - 1) / lenk;   // chunks of dim k (the last outer dim, possibly 1)
+    bd->out_ext[no] = int32_t(nch);
+    bd->out_g[no] = int32_t(gst[k] * lenk);
+    magic32(nch, &bd->out_mul[no], &bd->out_shift[no]);
+    for (int a = 0; a < ra; ++a) bd->out_c[no][ra - 1 - a] = int32_t((int64_t(td.coef[a][k]) * lenk) % td.ashape[a]);
+    ++no;
+    bd->n_out = no;
+    int64_t nblocks = nch;
+    for (int d = 0; d < k; ++d) nblocks *= td.ext[d];
+    if (nblocks >= (int64_t(1) << 31)) return false;
+    bd->nblocks = int32_t(nblocks);
+    bd->n_in = nd - k;
+    bd->chunk_ext = int32_t(td.ext[k]);
+    bd->chunk_len = int32_t(lenk);
+    for (int j = 0; j < bd->n_in; ++j) {
+        const int d = k + j;
+        bd->in_len[j] = int32_t(j == 0 ? lenk : td.ext[d]);
+        for (int a = 0; a < ra; ++a) bd->in_c[j][ra - 1 - a] = int32_t(sc[d][a]);
+        if (j >= 1) magic32(td.ext[d], &bd->in_mul[j], &bd->in_shift[j]);
+    }
+    bd->tail_prod = int32_t(inner / lenk);
+    magic32(bd->tail_prod, &bd->tail_mul, &bd->tail_shift);
+    bd->pitch_pad = (E[ra - 1] % 32 == 0) ? 1 : 0;   // rows of 32-multiple length: odd pitch, fewer bank conflicts
+    const int64_t rows = vol / E[ra - 1];
+    *smem_bytes = int(rows * (E[ra - 1] + bd->pitch_pad) * es);
+    return true;
+}
+
+// AOL_TILER_BOX=0 disables the staged box kernels (A/B measurements only).
+bool tiler_box_enabled() {
+    static const bool v = [] {
+        const char* e = std::getenv("AOL_TILER_BOX");
+        return !(e && e[0] == '0');
+    }();
+    return v;
+}
+
 // AOL_TILER_WRAPTAB=0 runs wrapping gathers / FAST scatters element by element (A/B measurements only).
 bool tiler_wraptab_enabled() {
     static const bool v = [] {
@@ -825,6 +1188,27 @@ aol_status_t launch_v(const TilerDev& td, const void* src, void* dst, unsigned l
         return AOL_OK;
     }
     if constexpr (V == 1) {
+        BoxDev bd;
+        int box_smem = 0;
+        if (MODE <= 1 && !lin && tiler_box_enabled() && make_box(td, ES, MODE, &bd, &box_smem)) {
+          if constexpr (MODE <= 1) {
+            DeviceInfo dev;
+            aol_status_t st = device_info(&dev);
+            if (st != AOL_OK) return st;
+            // 16-byte vectors on the tile side when every block starts and ends on a 16-byte boundary
+            constexpr int VW = 16 / ES;
+            const void* tp = MODE == 0 ? dst : src;
+            bool vec = reinterpret_cast<uintptr_t>(tp) % 16 == 0 && (int64_t(bd.tail_prod) * ES) % 16 == 0;
+            for (int d = 0; d < bd.n_out && vec; ++d) vec = (int64_t(bd.out_g[d]) * ES) % 16 == 0;
+            const int gb = int(std::max<int64_t>(1, std::min<int64_t>(bd.nblocks, int64_t(dev.num_sms) * 4)));
+            if (vec)
+                tiler_box_kernel<ES, VW, MODE><<<gb, 256, box_smem, s>>>(bd, src, dst);
+            else
+                tiler_box_kernel<ES, 1, MODE><<<gb, 256, box_smem, s>>>(bd, src, dst);
+            AOL_LAUNCH_CHECK("tiler_box_kernel");
+            return AOL_OK;
+          }
+        }
         Wrap32Dev wd;
         if (!lin && tiler_wrap32_enabled() && make_wrap32(td, &wd)) {
             DeviceInfo dev;
