@@ -377,7 +377,8 @@ aol_status_t enqueue_fused(const FusedLaunch& L, uint64_t* d_cs, cudaStream_t s)
     // for its own predecessor); pdl therefore requires d_cs, and the zero kernel is launched right before it.
     // cs_mode 1 (plans) needs no zeroing: one launch.
     const bool zero = d_cs && a.cs_mode == 0;
-    const bool pdl = zero && !(L.flags & AOL_FLAG_NO_PDL);
+    // cs_mode 0: PDL after the zeroing kernel; plans (pdl_wait): PDL after whatever precedes (the kernel waits)
+    const bool pdl = (zero || a.pdl_wait) && !(L.flags & AOL_FLAG_NO_PDL);
     if (zero) {
         cudaLaunchConfig_t zc;
         std::memset(&zc, 0, sizeof zc);

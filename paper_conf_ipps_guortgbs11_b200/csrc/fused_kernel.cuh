@@ -122,6 +122,9 @@ struct FusedArgs {
     // cs_partial[unit] and counts itself in cs_count[frame]; the frame's last unit sums the partials into
     // cs[frame] and resets the counter to 0 for the next launch (self-resetting, one launch per call).
     int32_t cs_mode;
+    int32_t pdl_wait;           // 1: launched as a programmatic dependent of an ARBITRARY predecessor (plans): the
+                                // producer and consumer thread 0 -- the only threads touching global memory --
+                                // wait for it (griddepcontrol.wait) before their first access
     int32_t units_per_frame;    // cs_mode 1: work units of one frame (contiguous unit indices)
     unsigned long long* cs_partial;
     unsigned int* cs_count;
@@ -234,7 +237,18 @@ __device__ __forceinline__ void h_row(uint32_t row_base, uint32_t rr, const RepG
             x[2] = uint32_t(v.z);
             x[3] = uint32_t(v.w);
         }
-        x[2 * kR] = ptx::lds32(rowa + g.offn);
+#ifdef AOL_U8_NBR_LDS
+        x[2 * kR] = ptx::lds32(rowa + g.offn);   // A/B build: every lane loads the neighbour word (bank conflicts)
+#else
+        // the next repetition's first word is lane+1's x[0]: one shuffle (an LDS.32 at the 8kR-byte lane stride
+        // was a 2-way (kR = 1) / 4-way (kR = 2) bank conflict); lane 31 and the row-wrapping repetition load it
+        {
+            uint32_t nw = __shfl_down_sync(0xffffffffu, x[0], 1);
+            uint32_t nl = 0;
+            ptx::lds32_if(nl, rowa + g.offn, g.fix);
+            x[2 * kR] = g.fix ? nl : nw;
+        }
+#endif
 #pragma unroll
         for (int j = 0; j < kR; ++j) {
             const uint32_t lo = x[2 * j], hi = x[2 * j + 1], nw = x[2 * j + 2];
@@ -288,6 +302,7 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
         // ------------------------------------------------ producer warp (TMA)
         if (tid == NC) {
             if ((kI32 && kSwz != 0) || a.u8_tensor) ptx::prefetch_tensormap(&tmap);
+            if (a.pdl_wait) ptx::griddep_wait();
             int s = 0;
             uint32_t ph = 0;
             for (int64_t k = 0, u = unit_of(a, 0); u < a.nunits; u = unit_of(a, ++k)) {
@@ -347,6 +362,7 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
     }
 
     // ---------------------------------------------------- consumer threads
+    if (a.pdl_wait && tid == 0) ptx::griddep_wait();
     const int lane = tid & 31;
     const bool active = kRP * tid < a.reps;
     const int r = active ? kRP * tid : a.reps - kRP;   // first repetition owned (clamped for idle lanes)
@@ -377,7 +393,7 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
         g.off0 = 8u * uint32_t(r);
         g.off1 = g.off0 + 4;
         g.offn = 8u * uint32_t(rn);
-        g.fix = false;
+        g.fix = (lane == 31) || (r + kRP == a.reps);   // neighbour word not in lane+1 (see h_row)
     }
     const uint32_t segs = uint32_t(a.segs);
     const uint32_t Wu = uint32_t(a.W);
@@ -593,27 +609,37 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
             for (int off = 16; off > 0; off >>= 1) csacc += __shfl_xor_sync(0xffffffffu, csacc, off);
             if (lane == 0) red[tid >> 5] = csacc;
             ptx::named_bar_sync(2, NC);
-            if (tid == 0) {
+            if (tid < 32) {   // warp 0
                 unsigned long long sum = 0;
-                for (int w = 0; w < NC / 32; ++w) sum += red[w];
+                if (lane == 0)
+                    for (int w = 0; w < NC / 32; ++w) sum += red[w];
                 const int64_t frame = plane / a.channels;
                 if (a.cs_mode == 0) {
                     // the checksums were zeroed by the preceding zero_checksums_kernel, which this launch may
                     // overlap (programmatic dependent launch): wait for it before the first atomic (no-op when
                     // the kernel was launched without the PDL attribute, and after the first wait)
-                    ptx::griddep_wait();
-                    atomicAdd(reinterpret_cast<unsigned long long*>(a.cs + frame), sum);
+                    if (lane == 0) {
+                        ptx::griddep_wait();
+                        atomicAdd(reinterpret_cast<unsigned long long*>(a.cs + frame), sum);
+                    }
                 } else {
-                    a.cs_partial[u] = sum;
-                    __threadfence();   // the partial is visible before the count that publishes it
-                    const unsigned prev = atomicAdd(a.cs_count + frame, 1u);
-                    if (prev == unsigned(a.units_per_frame - 1)) {   // the frame's last unit
+                    unsigned last = 0;
+                    if (lane == 0) {
+                        a.cs_partial[u] = sum;
+                        __threadfence();   // the partial is visible before the count that publishes it
+                        last = atomicAdd(a.cs_count + frame, 1u) == unsigned(a.units_per_frame - 1) ? 1u : 0u;
+                    }
+                    if (__shfl_sync(0xffffffffu, last, 0)) {   // the frame's last unit: sum its partials
                         __threadfence();
                         const int64_t u0 = frame * a.units_per_frame;
                         unsigned long long tot = 0;
-                        for (int32_t j = 0; j < a.units_per_frame; ++j) tot += __ldcg(a.cs_partial + u0 + j);
-                        a.cs[frame] = tot;
-                        a.cs_count[frame] = 0u;   // ready for the next launch (stream-ordered after this grid)
+                        for (int32_t j = lane; j < a.units_per_frame; j += 32) tot += __ldcg(a.cs_partial + u0 + j);
+#pragma unroll
+                        for (int off = 16; off > 0; off >>= 1) tot += __shfl_xor_sync(0xffffffffu, tot, off);
+                        if (lane == 0) {
+                            a.cs[frame] = tot;
+                            a.cs_count[frame] = 0u;   // ready for the next launch (stream-ordered after this grid)
+                        }
                     }
                 }
             }

@@ -65,6 +65,7 @@ aol_status_t aol_frame_plan_create(const void* d_in, aol_dtype_t in_dtype, void*
                 st = AOL_E_CUDA;
             } else {
                 p->launch.args.cs_mode = 1;
+                p->launch.args.pdl_wait = 1;
                 p->launch.args.cs_partial = static_cast<unsigned long long*>(p->d_ws);
                 p->launch.args.cs_count = reinterpret_cast<unsigned int*>(static_cast<uint8_t*>(p->d_ws) + units * 8);
             }

@@ -562,7 +562,8 @@ WrapTabDev make_wraptab(const Wrap32Dev& wd) {
 // tilers, ArrayOL single assignment).  Replaces the per-element offset arithmetic of the kernels above with
 // ~10 instructions per element and keeps both global sides streaming.
 constexpr int kBoxMaxInner = 4;           // inner dims (incl. the chunked one)
-constexpr int kBoxBytes = 48 * 1024;      // smem box per CTA (4 CTAs per SM)
+constexpr int kBoxBytes = 40 * 1024;      // smem box per CTA (+ the offset table: 2-4 CTAs per SM)
+constexpr int kBoxTab = 8192;             // entries of the per-CTA inner offset table (32 KB)
 
 // Array dims are stored REVERSED in the box descriptors (r = 0 is the innermost, contiguous array dim: the box
 // row), so that every per-dim array is indexed by compile-time constants after unrolling (registers, no local
@@ -679,52 +680,45 @@ __device__ __forceinline__ int32_t box_row_offset(const BoxDev& bd, const BoxBlo
     return off;
 }
 
-// Smem offset of the box element holding inner element e of the block (e < count).
-__device__ __forceinline__ int32_t box_inner_offset(const BoxDev& bd, const BoxBlock& b, uint32_t e,
-                                                    int32_t (&idx)[kBoxMaxInner]) {
-    const uint32_t i0 = magic_div(e, bd.tail_mul, bd.tail_shift);
-    uint32_t rem = e - i0 * uint32_t(bd.tail_prod);
-    idx[0] = int32_t(i0);
-    int32_t off = b.off0 + b.step[0] * int32_t(i0);
+// Smem offsets of the TAIL of the inner block (inner dims >= 1, tail_prod elements, row-major) relative to the
+// offset of its inner-dim-0 index: tab[t] = sum_{d >= 1} step[d] idx_d(t).  Built per CTA whenever the box
+// layout changes (only between a full and the ragged last chunk), so an element's box offset is then
+// off0 + step[0] i0 + tab[t]: one magic division per 16-byte vector and two shared loads per element.
+__device__ __forceinline__ void box_build_table(const BoxDev& bd, const BoxBlock& b, int32_t* tab) {
+    for (int32_t t = threadIdx.x; t < bd.tail_prod; t += blockDim.x) {
+        uint32_t rem = uint32_t(t);
+        int32_t off = 0;
 #pragma unroll
-    for (int d = kBoxMaxInner - 1; d >= 1; --d) {
-        if (d >= bd.n_in) continue;
-        const uint32_t q = magic_div(rem, bd.in_mul[d], bd.in_shift[d]);
-        const int32_t i = int32_t(rem - q * uint32_t(bd.in_len[d]));
-        rem = q;
-        idx[d] = i;
-        off += b.step[d] * i;
-    }
-    return off;
-}
-
-// Advance the inner index by one (odometer over the inner dims, innermost last).
-__device__ __forceinline__ void box_inner_next(const BoxDev& bd, const BoxBlock& b, int32_t (&idx)[kBoxMaxInner],
-                                               int32_t& off) {
-#pragma unroll
-    for (int d = kBoxMaxInner - 1; d >= 0; --d) {
-        if (d >= bd.n_in) continue;
-        const int32_t len = d == 0 ? b.len0 : bd.in_len[d];
-        off += b.step[d];
-        if (++idx[d] < len) return;
-        idx[d] = 0;
-        off -= b.step[d] * len;
+        for (int d = kBoxMaxInner - 1; d >= 1; --d) {
+            if (d >= bd.n_in) continue;
+            const uint32_t q = magic_div(rem, bd.in_mul[d], bd.in_shift[d]);
+            off += b.step[d] * int32_t(rem - q * uint32_t(bd.in_len[d]));
+            rem = q;
+        }
+        tab[t] = off;
     }
 }
 
+// smem: [tail_prod] int32 offset table, then the box (16-byte aligned).
 template <int ES, int VW, int MODE>
 __global__ void __launch_bounds__(256) tiler_box_kernel(const __grid_constant__ BoxDev bd, const void* __restrict__ src,
                                                         void* __restrict__ dst) {
     using T = typename Elem<ES>::T;
     using VT = typename Vec<ES * VW>::T;
     extern __shared__ __align__(16) uint8_t box_raw[];
-    T* box = reinterpret_cast<T*>(box_raw);
+    int32_t* tab = reinterpret_cast<int32_t*>(box_raw);
+    T* box = reinterpret_cast<T*>(box_raw + ((size_t(bd.tail_prod) * 4 + 15) & ~size_t(15)));
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
     const int sl = bd.ashape[0];
+    int32_t tab_len0 = -1;   // len0 the table was built for
     for (int32_t blk = blockIdx.x; blk < bd.nblocks; blk += gridDim.x) {
         BoxBlock b;
         box_block(bd, blk, b);
         const int32_t El = b.E[0], c0 = b.base[0];
+        if (b.len0 != tab_len0) {   // uniform across the CTA; the previous block's reads of tab have finished
+            box_build_table(bd, b, tab);
+            tab_len0 = b.len0;
+        }
         if (MODE == 0) {
             // ---- load the box: a warp per row, lanes along the row (coalesced), wrap at the row's end
             const T* A = static_cast<const T*>(src);
@@ -750,30 +744,28 @@ __global__ void __launch_bounds__(256) tiler_box_kernel(const __grid_constant__ 
             // ---- write the tile block: VW consecutive tile elements per thread (16-byte stores)
             T* Tg = static_cast<T*>(dst) + b.g0;
             for (int32_t v = threadIdx.x; v * VW < b.count; v += 256) {
-                int32_t idx[kBoxMaxInner] = {0, 0, 0, 0};
-                int32_t off = box_inner_offset(bd, b, uint32_t(v * VW), idx);
+                const uint32_t e = uint32_t(v * VW);
+                const uint32_t i0 = magic_div(e, bd.tail_mul, bd.tail_shift);
+                const int32_t t = int32_t(e - i0 * uint32_t(bd.tail_prod));
+                const int32_t o = b.off0 + b.step[0] * int32_t(i0);
                 union { VT vec; T e[VW]; } pk;
 #pragma unroll
-                for (int j = 0; j < VW; ++j) {
-                    pk.e[j] = box[off];
-                    if (j + 1 < VW) box_inner_next(bd, b, idx, off);
-                }
+                for (int j = 0; j < VW; ++j) pk.e[j] = box[o + tab[t + j]];
                 reinterpret_cast<VT*>(Tg)[v] = pk.vec;
             }
-            __syncthreads();   // the box is reloaded by the next block
+            __syncthreads();   // the box (and tab) are rewritten by the next block
         } else {
             // ---- FAST scatter: the tile block into the box (it covers the box exactly), then the box out
             const T* Tg = static_cast<const T*>(src) + b.g0;
             for (int32_t v = threadIdx.x; v * VW < b.count; v += 256) {
                 union { VT vec; T e[VW]; } pk;
                 pk.vec = reinterpret_cast<const VT*>(Tg)[v];
-                int32_t idx[kBoxMaxInner] = {0, 0, 0, 0};
-                int32_t off = box_inner_offset(bd, b, uint32_t(v * VW), idx);
+                const uint32_t e = uint32_t(v * VW);
+                const uint32_t i0 = magic_div(e, bd.tail_mul, bd.tail_shift);
+                const int32_t t = int32_t(e - i0 * uint32_t(bd.tail_prod));
+                const int32_t o = b.off0 + b.step[0] * int32_t(i0);
 #pragma unroll
-                for (int j = 0; j < VW; ++j) {
-                    box[off] = pk.e[j];
-                    if (j + 1 < VW) box_inner_next(bd, b, idx, off);
-                }
+                for (int j = 0; j < VW; ++j) box[o + tab[t + j]] = pk.e[j];
             }
             __syncthreads();
             T* A = static_cast<T*>(dst);
@@ -830,6 +822,9 @@ bool make_box(const TilerDev& td, int es, int mode, BoxDev* bd, int* smem_bytes)
         if (vol + pitch_extra * (vol / std::max<int64_t>(1, E[ra - 1])) <= budget) {   // all of dim k fits
             lenk = td.ext[k];
             if (k == 0 || nd - (k - 1) > kBoxMaxInner) break;
+            int64_t tail = 1;   // the table would cover dims k..nd-1 once dim k-1 is the chunked one
+            for (int d = k; d < nd; ++d) tail *= td.ext[d];
+            if (tail > kBoxTab) break;
             int64_t E2[AOL_MAX_RANK];
             const int64_t v2 = box_of(k - 1, 1, E2);   // would one slice of dim k-1 still fit?
             if (v2 + pitch_extra * (v2 / std::max<int64_t>(1, E2[ra - 1])) > budget) break;
@@ -852,6 +847,7 @@ bool make_box(const TilerDev& td, int es, int mode, BoxDev* bd, int* smem_bytes)
     const int64_t vol = box_of(k, lenk, E);
     int64_t inner = lenk;
     for (int d = k + 1; d < nd; ++d) inner *= td.ext[d];
+    if (inner / lenk > kBoxTab) return false;
     if (mode == 0 ? (2 * vol > 3 * inner) : (vol != inner)) return false;
     if (E[ra - 1] < 32) return false;
     if (E[ra - 1] > 2 * td.ashape[ra - 1]) return false;   // the row wrap takes at most two subtractions
@@ -898,7 +894,7 @@ bool make_box(const TilerDev& td, int es, int mode, BoxDev* bd, int* smem_bytes)
     magic32(bd->tail_prod, &bd->tail_mul, &bd->tail_shift);
     bd->pitch_pad = (E[ra - 1] % 32 == 0) ? 1 : 0;   // rows of 32-multiple length: odd pitch, fewer bank conflicts
     const int64_t rows = vol / E[ra - 1];
-    *smem_bytes = int(rows * (E[ra - 1] + bd->pitch_pad) * es);
+    *smem_bytes = int(((inner / lenk) * 4 + 15) / 16 * 16 + rows * (E[ra - 1] + bd->pitch_pad) * es);
     return true;
 }
 
