@@ -237,11 +237,13 @@ __device__ __forceinline__ void h_row(uint32_t row_base, uint32_t rr, const RepG
             x[2] = uint32_t(v.z);
             x[3] = uint32_t(v.w);
         }
-#ifdef AOL_U8_NBR_LDS
-        x[2 * kR] = ptx::lds32(rowa + g.offn);   // A/B build: every lane loads the neighbour word (bank conflicts)
+#ifndef AOL_U8_NBR_SHFL
+        // the next repetition's first word by one LDS.32 per lane: at the 8kR-byte lane stride a 2-way (kR = 1) /
+        // 4-way (kR = 2) bank conflict, but the kernel is issue-bound, not LSU-bound: a shuffle plus a predicated
+        // LDS for lane 31 removes the conflicts and costs 16 M more instructions, 2 % slower
+        // (profiles/r02_u8_nbr_ab.jsonl; A/B build flag AOL_U8_NBR_SHFL)
+        x[2 * kR] = ptx::lds32(rowa + g.offn);
 #else
-        // the next repetition's first word is lane+1's x[0]: one shuffle (an LDS.32 at the 8kR-byte lane stride
-        // was a 2-way (kR = 1) / 4-way (kR = 2) bank conflict); lane 31 and the row-wrapping repetition load it
         {
             uint32_t nw = __shfl_down_sync(0xffffffffu, x[0], 1);
             uint32_t nl = 0;

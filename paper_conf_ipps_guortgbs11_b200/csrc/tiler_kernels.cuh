@@ -1196,11 +1196,12 @@ aol_status_t launch_v(const TilerDev& td, const void* src, void* dst, unsigned l
             const void* tp = MODE == 0 ? dst : src;
             bool vec = reinterpret_cast<uintptr_t>(tp) % 16 == 0 && (int64_t(bd.tail_prod) * ES) % 16 == 0;
             for (int d = 0; d < bd.n_out && vec; ++d) vec = (int64_t(bd.out_g[d]) * ES) % 16 == 0;
-            const int gb = int(std::max<int64_t>(1, std::min<int64_t>(bd.nblocks, int64_t(dev.num_sms) * 4)));
-            if (vec)
-                tiler_box_kernel<ES, VW, MODE><<<gb, 256, box_smem, s>>>(bd, src, dst);
-            else
-                tiler_box_kernel<ES, 1, MODE><<<gb, 256, box_smem, s>>>(bd, src, dst);
+            auto kern = vec ? tiler_box_kernel<ES, VW, MODE> : tiler_box_kernel<ES, 1, MODE>;
+            st = kernel_smem(reinterpret_cast<const void*>(kern), box_smem);   // up to 72 KB (table + box)
+            if (st != AOL_OK) return st;
+            const int per_sm = std::max(1, kernel_occupancy(reinterpret_cast<const void*>(kern), 256, box_smem));
+            const int gb = int(std::max<int64_t>(1, std::min<int64_t>(bd.nblocks, int64_t(dev.num_sms) * per_sm)));
+            kern<<<gb, 256, box_smem, s>>>(bd, src, dst);
             AOL_LAUNCH_CHECK("tiler_box_kernel");
             return AOL_OK;
           }
