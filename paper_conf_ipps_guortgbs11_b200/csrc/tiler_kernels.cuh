@@ -28,6 +28,7 @@
 #include <cstring>
 
 #include "common.h"
+#include "ptx.cuh"
 
 namespace aol {
 
@@ -562,7 +563,7 @@ WrapTabDev make_wraptab(const Wrap32Dev& wd) {
 // tilers, ArrayOL single assignment).  Replaces the per-element offset arithmetic of the kernels above with
 // ~10 instructions per element and keeps both global sides streaming.
 constexpr int kBoxMaxInner = 4;           // inner dims (incl. the chunked one)
-constexpr int kBoxBytes = 40 * 1024;      // smem box per CTA (+ the offset table: 2-4 CTAs per SM)
+constexpr int kBoxBytes = 36 * 1024;      // smem per box buffer (gather: two, + the offset table: 2 CTAs per SM)
 constexpr int kBoxTab = 8192;             // entries of the per-CTA inner offset table (32 KB)
 
 // Array dims are stored REVERSED in the box descriptors (r = 0 is the innermost, contiguous array dim: the box
@@ -699,49 +700,84 @@ __device__ __forceinline__ void box_build_table(const BoxDev& bd, const BoxBlock
     }
 }
 
-// smem: [tail_prod] int32 offset table, then the box (16-byte aligned).
+// Issue the loads of a block's box into smem buffer `buf`: a warp per box row, lanes along the row (coalesced),
+// wrapped at the row's end.  4- and 8-byte elements: asynchronous copies (cp.async, committed as one group by
+// the caller: the whole box in flight at once); 1- and 2-byte elements: plain loads and stores.
+template <int ES>
+__device__ __forceinline__ void box_issue_load(const BoxDev& bd, const BoxBlock& b, const void* src, uint8_t* buf) {
+    using T = typename Elem<ES>::T;
+    const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+    const int sl = bd.ashape[0];
+    const int32_t El = b.E[0], c0 = b.base[0];
+    const T* A = static_cast<const T*>(src);
+    for (int32_t row = warp; row < b.rows; row += 8) {
+        const int32_t roff = box_row_offset(bd, b, row);
+        if constexpr (ES >= 4) {
+            const uint32_t srow = ptx::smem_u32(buf) + uint32_t(row * b.pitch) * ES;
+            for (int32_t x = lane; x < El; x += 32) {
+                int32_t gc = c0 + x;
+                while (gc >= sl) gc -= sl;
+                ptx::cp_async<ES>(srow + uint32_t(x) * ES, A + roff + gc);
+            }
+        } else {
+            T* srow = reinterpret_cast<T*>(buf) + row * b.pitch;
+            constexpr int kU = 8;
+            for (int32_t x0 = lane; x0 < El; x0 += 32 * kU) {
+                T v[kU];
+#pragma unroll
+                for (int u = 0; u < kU; ++u) {
+                    const int32_t x = x0 + 32 * u;
+                    int32_t gc = c0 + x;
+                    while (gc >= sl) gc -= sl;
+                    if (x < El) v[u] = A[roff + gc];
+                }
+#pragma unroll
+                for (int u = 0; u < kU; ++u)
+                    if (x0 + 32 * u < El) srow[x0 + 32 * u] = v[u];
+            }
+        }
+    }
+}
+
+// smem: [tail_prod] int32 offset table, then one box buffer (FAST scatter) or two (gather: the next block's box
+// loads asynchronously while the current one is written out), each 16-byte aligned.
 template <int ES, int VW, int MODE>
 __global__ void __launch_bounds__(256) tiler_box_kernel(const __grid_constant__ BoxDev bd, const void* __restrict__ src,
-                                                        void* __restrict__ dst) {
+                                                        void* __restrict__ dst, int32_t buf_bytes) {
     using T = typename Elem<ES>::T;
     using VT = typename Vec<ES * VW>::T;
     extern __shared__ __align__(16) uint8_t box_raw[];
     int32_t* tab = reinterpret_cast<int32_t*>(box_raw);
-    T* box = reinterpret_cast<T*>(box_raw + ((size_t(bd.tail_prod) * 4 + 15) & ~size_t(15)));
+    uint8_t* bufs = box_raw + ((size_t(bd.tail_prod) * 4 + 15) & ~size_t(15));
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
     const int sl = bd.ashape[0];
     int32_t tab_len0 = -1;   // len0 the table was built for
-    for (int32_t blk = blockIdx.x; blk < bd.nblocks; blk += gridDim.x) {
-        BoxBlock b;
-        box_block(bd, blk, b);
-        const int32_t El = b.E[0], c0 = b.base[0];
-        if (b.len0 != tab_len0) {   // uniform across the CTA; the previous block's reads of tab have finished
-            box_build_table(bd, b, tab);
-            tab_len0 = b.len0;
+    if (MODE == 0) {
+        // software pipeline over this CTA's blocks: box k+1 loads while box k is emitted
+        int32_t blk = blockIdx.x;
+        if (blk < bd.nblocks) {
+            BoxBlock b;
+            box_block(bd, blk, b);
+            box_issue_load<ES>(bd, b, src, bufs);
         }
-        if (MODE == 0) {
-            // ---- load the box: a warp per row, lanes along the row (coalesced), wrap at the row's end
-            const T* A = static_cast<const T*>(src);
-            for (int32_t row = warp; row < b.rows; row += 8) {
-                const int32_t roff = box_row_offset(bd, b, row);
-                T* srow = box + row * b.pitch;
-                constexpr int kU = 4;
-                for (int32_t x0 = lane; x0 < El; x0 += 32 * kU) {
-                    T v[kU];
-#pragma unroll
-                    for (int u = 0; u < kU; ++u) {
-                        const int32_t x = x0 + 32 * u;
-                        int32_t gc = c0 + x;
-                        while (gc >= sl) gc -= sl;
-                        if (x < El) v[u] = A[roff + gc];
-                    }
-#pragma unroll
-                    for (int u = 0; u < kU; ++u)
-                        if (x0 + 32 * u < El) srow[x0 + 32 * u] = v[u];
-                }
+        ptx::cp_async_commit();
+        for (int32_t k = 0; blk < bd.nblocks; ++k, blk += gridDim.x) {
+            const int32_t nxt = blk + gridDim.x;
+            if (nxt < bd.nblocks) {
+                BoxBlock bn;
+                box_block(bd, nxt, bn);
+                box_issue_load<ES>(bd, bn, src, bufs + ((k + 1) & 1) * buf_bytes);
             }
+            ptx::cp_async_commit();
+            BoxBlock b;
+            box_block(bd, blk, b);
+            if (b.len0 != tab_len0) {   // uniform across the CTA; the previous block's reads of tab have finished
+                box_build_table(bd, b, tab);
+                tab_len0 = b.len0;
+            }
+            ptx::cp_async_wait<1>();   // this block's box has landed (the next one may still be in flight)
             __syncthreads();
-            // ---- write the tile block: VW consecutive tile elements per thread (16-byte stores)
+            const T* box = reinterpret_cast<const T*>(bufs + (k & 1) * buf_bytes);
             T* Tg = static_cast<T*>(dst) + b.g0;
             for (int32_t v = threadIdx.x; v * VW < b.count; v += 256) {
                 const uint32_t e = uint32_t(v * VW);
@@ -753,19 +789,40 @@ __global__ void __launch_bounds__(256) tiler_box_kernel(const __grid_constant__ 
                 for (int j = 0; j < VW; ++j) pk.e[j] = box[o + tab[t + j]];
                 reinterpret_cast<VT*>(Tg)[v] = pk.vec;
             }
-            __syncthreads();   // the box (and tab) are rewritten by the next block
-        } else {
-            // ---- FAST scatter: the tile block into the box (it covers the box exactly), then the box out
+            __syncthreads();   // this buffer (and tab) may be overwritten from the next iteration on
+        }
+        ptx::cp_async_wait<0>();
+    } else {
+        T* box = reinterpret_cast<T*>(bufs);
+        for (int32_t blk = blockIdx.x; blk < bd.nblocks; blk += gridDim.x) {
+            BoxBlock b;
+            box_block(bd, blk, b);
+            const int32_t El = b.E[0], c0 = b.base[0];
+            if (b.len0 != tab_len0) {
+                box_build_table(bd, b, tab);
+                tab_len0 = b.len0;
+                __syncthreads();
+            }
+            // ---- FAST scatter: the tile block into the box (it covers the box exactly), then the box out;
+            // four 16-byte tile loads in flight per thread
             const T* Tg = static_cast<const T*>(src) + b.g0;
-            for (int32_t v = threadIdx.x; v * VW < b.count; v += 256) {
-                union { VT vec; T e[VW]; } pk;
-                pk.vec = reinterpret_cast<const VT*>(Tg)[v];
-                const uint32_t e = uint32_t(v * VW);
-                const uint32_t i0 = magic_div(e, bd.tail_mul, bd.tail_shift);
-                const int32_t t = int32_t(e - i0 * uint32_t(bd.tail_prod));
-                const int32_t o = b.off0 + b.step[0] * int32_t(i0);
+            constexpr int kU = 4;
+            for (int32_t v0 = threadIdx.x; v0 * VW < b.count; v0 += 256 * kU) {
+                union { VT vec; T e[VW]; } pk[kU];
 #pragma unroll
-                for (int j = 0; j < VW; ++j) box[o + tab[t + j]] = pk.e[j];
+                for (int u = 0; u < kU; ++u)
+                    if ((v0 + 256 * u) * VW < b.count) pk[u].vec = reinterpret_cast<const VT*>(Tg)[v0 + 256 * u];
+#pragma unroll
+                for (int u = 0; u < kU; ++u) {
+                    const int32_t v = v0 + 256 * u;
+                    if (v * VW >= b.count) continue;
+                    const uint32_t e = uint32_t(v * VW);
+                    const uint32_t i0 = magic_div(e, bd.tail_mul, bd.tail_shift);
+                    const int32_t t = int32_t(e - i0 * uint32_t(bd.tail_prod));
+                    const int32_t o = b.off0 + b.step[0] * int32_t(i0);
+#pragma unroll
+                    for (int j = 0; j < VW; ++j) box[o + tab[t + j]] = pk[u].e[j];
+                }
             }
             __syncthreads();
             T* A = static_cast<T*>(dst);
@@ -786,7 +843,7 @@ __global__ void __launch_bounds__(256) tiler_box_kernel(const __grid_constant__ 
 // Plan the box form of a tiler (fast32, every offset < 2^31); false if it does not qualify: the inner block
 // must be dense in its box (gather: box <= 1.5 x inner elements; scatter: exactly equal), box rows >= 32
 // elements long, <= kBoxMaxInner inner dims, box within kBoxBytes.
-bool make_box(const TilerDev& td, int es, int mode, BoxDev* bd, int* smem_bytes) {
+bool make_box(const TilerDev& td, int es, int mode, BoxDev* bd, int* smem_bytes, int* buf_bytes) {
     if (!td.fast32 || td.array_elems >= (int64_t(1) << 31) || td.nd == 0) return false;
     std::memset(bd, 0, sizeof *bd);
     const int nd = td.nd, ra = td.ra;
@@ -894,7 +951,9 @@ bool make_box(const TilerDev& td, int es, int mode, BoxDev* bd, int* smem_bytes)
     magic32(bd->tail_prod, &bd->tail_mul, &bd->tail_shift);
     bd->pitch_pad = (E[ra - 1] % 32 == 0) ? 1 : 0;   // rows of 32-multiple length: odd pitch, fewer bank conflicts
     const int64_t rows = vol / E[ra - 1];
-    *smem_bytes = int(((inner / lenk) * 4 + 15) / 16 * 16 + rows * (E[ra - 1] + bd->pitch_pad) * es);
+    const int64_t buf = (rows * (E[ra - 1] + bd->pitch_pad) * es + 15) / 16 * 16;
+    *buf_bytes = int(buf);
+    *smem_bytes = int(((inner / lenk) * 4 + 15) / 16 * 16 + (mode == 0 ? 2 : 1) * buf);
     return true;
 }
 
@@ -1185,8 +1244,8 @@ aol_status_t launch_v(const TilerDev& td, const void* src, void* dst, unsigned l
     }
     if constexpr (V == 1) {
         BoxDev bd;
-        int box_smem = 0;
-        if (MODE <= 1 && !lin && tiler_box_enabled() && make_box(td, ES, MODE, &bd, &box_smem)) {
+        int box_smem = 0, box_buf = 0;
+        if (MODE <= 1 && !lin && tiler_box_enabled() && make_box(td, ES, MODE, &bd, &box_smem, &box_buf)) {
           if constexpr (MODE <= 1) {
             DeviceInfo dev;
             aol_status_t st = device_info(&dev);
@@ -1201,7 +1260,7 @@ aol_status_t launch_v(const TilerDev& td, const void* src, void* dst, unsigned l
             if (st != AOL_OK) return st;
             const int per_sm = std::max(1, kernel_occupancy(reinterpret_cast<const void*>(kern), 256, box_smem));
             const int gb = int(std::max<int64_t>(1, std::min<int64_t>(bd.nblocks, int64_t(dev.num_sms) * per_sm)));
-            kern<<<gb, 256, box_smem, s>>>(bd, src, dst);
+            kern<<<gb, 256, box_smem, s>>>(bd, src, dst, box_buf);
             AOL_LAUNCH_CHECK("tiler_box_kernel");
             return AOL_OK;
           }
