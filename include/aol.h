@@ -327,6 +327,17 @@ AOL_API aol_status_t aol_filter_validate(const aol_filter_t* f);
  * (cells no repetition writes keep their value).  4-byte aligned.  Async on s. */
 AOL_API aol_status_t aol_filter_apply(const aol_filter_t* f, const int32_t* d_in, int32_t* d_out, cudaStream_t s);
 
+/* Two repetitions chained -- f2 consumes f1's output array -- in ONE kernel: d_out = f2(f1(d_in)), the
+ * intermediate array never stored (WITH-loop folding across repetitions, for run-time
+ * descriptors; the paper's generic filters ran as separate kernels with host-side tilers).
+ * Fused when f1's output tiler is a bijection onto its array whose window digits are the low digits of
+ * each dimension (the paper's H and V output tilers are), f2's output tiler does not wrap, ranks <= 4 and
+ * patterns <= 16 elements; otherwise the two filters run as two launches through d_workspace (>= the
+ * intermediate array's bytes; NULL -> AOL_E_WORKSPACE naming the reason).  f1.out.array_shape must equal
+ * f2.in.array_shape.  d_in / d_out int32 shaped f1.in / f2.out arrays, 4-byte aligned.  Async on s. */
+AOL_API aol_status_t aol_filter_chain_apply(const aol_filter_t* f1, const aol_filter_t* f2, const int32_t* d_in,
+                                            int32_t* d_out, void* d_workspace, size_t ws_bytes, cudaStream_t s);
+
 /* ------------------------------------------- synthetic input (test support) */
 
 /* Fill d_out [nframes][channels][H][W] with the counter-based synthetic frames

@@ -28,7 +28,7 @@ __all__ = [
     "tiler_gather", "tiler_scatter", "tiler_scatter_workspace_bytes", "downscale_h", "downscale_v", "downscale_frame", "downscale_frame_plan",
     "frame_checksum", "downscale_frame_host", "FramePlan", "synth_frames", "library_path", "downscale_frame_packed",
     "PRESET_H_IN", "PRESET_H_OUT", "PRESET_V_IN", "PRESET_V_OUT", "SYNTH_KINDS",
-    "make_filter", "filter_preset", "filter_validate", "filter_apply", "FILTER_H", "FILTER_V", "FLAGS",
+    "make_filter", "filter_preset", "filter_validate", "filter_apply", "filter_chain_apply", "last_kernel", "FILTER_H", "FILTER_V", "FLAGS",
 ]
 
 SYNTH_KINDS = {"uniform": 0, "dark": 1, "signed": 2, "ramp": 3, "constant": 4}
@@ -206,6 +206,27 @@ def filter_apply(f: aol_filter_t, x: torch.Tensor, out: Optional[torch.Tensor] =
     _out(out, a_out, torch.int32, x.device, "out")
     with torch.cuda.device(x.device):
         check(lib().aol_filter_apply(ctypes.byref(f), _dev(x, "x"), _dev(out, "out"), _stream(stream, x.device)))
+    return out
+
+
+def filter_chain_apply(f1: aol_filter_t, f2: aol_filter_t, x: torch.Tensor, out: Optional[torch.Tensor] = None,
+                       workspace: Optional[torch.Tensor] = None,
+                       stream: Optional[torch.cuda.Stream] = None) -> torch.Tensor:
+    """out = f2(f1(x)) in one fused kernel (the intermediate array never stored) when the chain qualifies,
+    else two launches through `workspace` (int32 tensor of f1's output array, or None -> error naming why)."""
+    a_in, _, _ = _shapes(f1.in_)
+    a_out, _, _ = _shapes(f2.out)
+    if x.dtype != torch.int32 or tuple(x.shape) != a_in:
+        raise ValueError(f"x must be int32 {a_in}")
+    if out is None:
+        out = torch.zeros(a_out, dtype=torch.int32, device=x.device)
+    _out(out, a_out, torch.int32, x.device, "out")
+    wp, wb = ctypes.c_void_p(0), 0
+    if workspace is not None:
+        wp, wb = _dev(workspace, "workspace"), workspace.numel() * workspace.element_size()
+    with torch.cuda.device(x.device):
+        check(lib().aol_filter_chain_apply(ctypes.byref(f1), ctypes.byref(f2), _dev(x, "x"), _dev(out, "out"), wp, wb,
+                                           _stream(stream, x.device)))
     return out
 
 

@@ -1,0 +1,749 @@
+// chain.cu -- NEXT row f3, fused: two run-time ArrayOL repetitions chained, f2 consuming f1's output array,
+// in ONE kernel -- WITH-loop folding across repetitions for descriptors known only at run time (the paper's
+// fusion, SaC WLF P:L528-546, applied to its generic formulation, Fig. 4-6, whose separately
+// launched generic filters it compares in Section VIII-A).  The intermediate array Y never
+// touches HBM.
+//
+// Work unit = a block of f2's repetitions (its inner repetition dims, the outermost of them in chunks).  The
+// block's pattern elements lie in a BOX of Y's raw coordinates (the footprint box of tiler_kernels.cuh).  A CTA
+//  (1) fills the box in shared memory by running f1 over exactly the f1 repetitions whose outputs land in it:
+//      f1's output tiler must be a bijection whose window digits are the low digits of each Y dim, so the
+//      repetitions covering a range of Y indices form a contiguous range per Y dim; each repetition gathers
+//      its pattern from X once (16-byte loads when it is a contiguous aligned run), forms its window sums from
+//      a shared-memory prefix array, applies the task and stores the outputs that fall inside the box;
+//  (2) runs f2 over the block's repetitions, their patterns read from the box, outputs stored to Z through
+//      f2's output tiler (linear: no wrap).
+// Anything outside these conditions runs as two aol_filter_apply launches through a caller workspace.
+#include <cuda_runtime.h>
+
+#include <algorithm>
+#include <cstdint>
+#include <cstdlib>
+#include <cstring>
+
+#include "common.h"
+
+namespace aol {
+namespace {
+
+constexpr int kCR = 4;       // array / repetition rank limit of the fused chain
+constexpr int kCP = 16;      // pattern elements per repetition
+constexpr int kCW = 16;      // windows per repetition
+constexpr int kCIn = 3;      // f2 inner repetition dims per block
+constexpr int kCDig = 3;     // digits of f1's output tiler per Y dim
+constexpr int kChainBox = 48 * 1024;   // smem bytes of the Y box
+
+struct ChainDev {
+    // ---------------- f1: X -> Y
+    int32_t rx, rr1;
+    int32_t sX[kCR], stX[kCR];
+    uint32_t mX_mul[kCR], mX_sh[kCR];          // floor(v / sX) for the reference point's mod
+    int32_t o1[kCR], P1[kCR][kCR];             // f1.in origin and paving, reduced mod sX  [a][j]
+    int32_t n_in1, len1, nwin1, div1;
+    uint32_t dv1_mul, dv1_sh;
+    int32_t start1[kCW];
+    int32_t f_in1[kCP][kCR], fmax_in1[kCR], lin_in1[kCP];
+    int32_t contig1, x_elems;
+    // f1's output tiler, per Y dim a: dense index v = (y - yo) mod sY = R K + kk; R's digits are f1 repetition
+    // indices (ascending, signed), kk(window) is a host table
+    int32_t ry;
+    int32_t sY[kCR], K[kCR], nRfull[kCR];       // nRfull = sY / K
+    int32_t yo[kCR];
+    int32_t nrd[kCR], rd_ext[kCR][kCDig], rd_neg[kCR][kCDig], rd_dim[kCR][kCDig];
+    int32_t kk[kCW][kCR];                        // window k's dense low part on each Y dim
+    // ---------------- f2: Y -> Z, blocked
+    int32_t rr2, n_in2, len2, nwin2, div2;
+    uint32_t dv2_mul, dv2_sh;
+    int32_t start2[kCW];
+    int32_t o2[kCR], P2[kCR][kCR];               // f2.in origin / paving mod sY  [a][j]
+    int32_t F2[kCP][kCR];                        // f2 pattern element p's signed raw offset on Y dim a
+    int32_t n_out, out_dim[kCR + 1], out_ext[kCR + 1], out_step[kCR + 1];   // outer rep dims (+ chunk index)
+    uint32_t out_mul[kCR + 1], out_sh[kCR + 1];
+    int32_t n_inr, in_dim[kCIn], in_len[kCIn];   // inner rep dims (0: chunked), full lengths
+    uint32_t in_mul[kCIn], in_sh[kCIn];
+    int32_t chunk_ext, chunk_len, tail_prod;
+    uint32_t tail_mul, tail_sh;
+    int32_t nblocks;
+    // f2's output tiler (linear): Z offset = zo + sum_j zP[j] r_j + zF[k]
+    int32_t zo, zP[kCR], zF[kCW];
+};
+
+__device__ __forceinline__ uint32_t mdiv(uint32_t n, uint32_t mul, uint32_t sh) { return (__umulhi(n, mul) + n) >> sh; }
+
+// C task: S/d - S%d (truncating), with |S| / |d| by a magic number.
+__device__ __forceinline__ int32_t task_c(int32_t S, int32_t d, uint32_t mul, uint32_t sh) {
+    const uint32_t qa = mdiv(uint32_t(abs(S)), mul, sh);
+    const int32_t q = ((S < 0) != (d < 0)) ? -int32_t(qa) : int32_t(qa);
+    return q * (1 + d) - S;
+}
+
+__global__ void __launch_bounds__(256) chain_kernel(const __grid_constant__ ChainDev cd, const int32_t* __restrict__ X,
+                                                    int32_t* __restrict__ Z) {
+    extern __shared__ __align__(16) int32_t sm[];
+    int32_t* pre = sm;                          // [kCP + 1][256] per-thread prefix sums
+    int32_t* poff = pre + (kCP + 1) * 256;      // [kCP] f2 pattern offsets in the box
+    int32_t* box = poff + kCP;
+    int32_t* my = pre + threadIdx.x;
+    for (int32_t blk = blockIdx.x; blk < cd.nblocks; blk += gridDim.x) {
+        // ---- block geometry: f2 outer repetition index, box over Y
+        int32_t r2[kCR];
+#pragma unroll
+        for (int j = 0; j < kCR; ++j) r2[j] = 0;
+        uint32_t n = uint32_t(blk);
+        int32_t ck = 0;
+        for (int d = cd.n_out - 1; d >= 0; --d) {
+            const uint32_t q = mdiv(n, cd.out_mul[d], cd.out_sh[d]);
+            const int32_t i = int32_t(n - q * uint32_t(cd.out_ext[d]));
+            n = q;
+            if (d == cd.n_out - 1) ck = i;
+            else {
+#pragma unroll
+                for (int j = 0; j < kCR; ++j)
+                    if (j == cd.out_dim[d]) r2[j] = i;
+            }
+        }
+        const int32_t len0 = min(cd.chunk_len, cd.chunk_ext - ck * cd.chunk_len);
+#pragma unroll
+        for (int j = 0; j < kCR; ++j)
+            if (j == cd.in_dim[0]) r2[j] = ck * cd.chunk_len;
+        // box extents / corner per Y dim (raw = o2 + P2 r2 + [lo, hi] over inner reps and pattern)
+        int32_t E[kCR], base[kCR], lo[kCR], bst[kCR];
+        int32_t rows = 1, pitch = 1, st = 1;
+#pragma unroll
+        for (int a = kCR - 1; a >= 0; --a) {
+            E[a] = 1;
+            base[a] = 0;
+            lo[a] = 0;
+            bst[a] = 0;
+            if (a >= cd.ry) continue;
+            int64_t raw = cd.o2[a];
+#pragma unroll
+            for (int j = 0; j < kCR; ++j)
+                if (j < cd.rr2) raw += int64_t(cd.P2[a][j]) * r2[j];
+            int32_t l = 0, h = 0;
+#pragma unroll
+            for (int d = 0; d < kCIn; ++d) {
+                if (d >= cd.n_inr) continue;
+                int32_t c = 0;
+#pragma unroll
+                for (int j = 0; j < kCR; ++j)
+                    if (j == cd.in_dim[d]) c = cd.P2[a][j];
+                if (2 * c > cd.sY[a]) c -= cd.sY[a];   // signed step
+                const int32_t ln = (d == 0 ? len0 : cd.in_len[d]) - 1;
+                if (c < 0) l += c * ln; else h += c * ln;
+            }
+            int32_t pl = 0, ph = 0;
+            for (int p = 0; p < cd.n_in2; ++p) {
+                pl = min(pl, cd.F2[p][a]);
+                ph = max(ph, cd.F2[p][a]);
+            }
+            l += pl;
+            h += ph;
+            E[a] = h - l + 1;
+            const int32_t v = int32_t((raw + l) % cd.sY[a]);
+            base[a] = v < 0 ? v + cd.sY[a] : v;
+            lo[a] = l;
+            bst[a] = st;
+            if (a == cd.ry - 1) {
+                pitch = E[a] + ((E[a] & 31) == 0 ? 1 : 0);
+                st = pitch;
+            } else {
+                st *= E[a];
+                rows *= E[a];
+            }
+        }
+        if (threadIdx.x < cd.n_in2) {
+            int32_t o = 0;
+#pragma unroll
+            for (int a = 0; a < kCR; ++a)
+                if (a < cd.ry) o += (cd.F2[threadIdx.x][a] - lo[a]) * bst[a];   // box offset of element p at r2
+            poff[threadIdx.x] = o;
+        }
+        // ---- (1) fill the box with f1: repetitions covering the box, a contiguous range of R per Y dim
+        int32_t R0[kCR], nR[kCR], v0[kCR];
+        int32_t nrep1 = 1;
+#pragma unroll
+        for (int a = 0; a < kCR; ++a) {
+            R0[a] = 0;
+            nR[a] = 1;
+            v0[a] = 0;
+            if (a >= cd.ry) continue;
+            int32_t v = base[a] - cd.yo[a];
+            if (v < 0) v += cd.sY[a];
+            v0[a] = v;
+            R0[a] = v / cd.K[a];
+            nR[a] = min((v + E[a] - 1) / cd.K[a] - R0[a] + 1, cd.nRfull[a] + 1);
+            nrep1 *= nR[a];
+        }
+        for (int32_t m = threadIdx.x; m < nrep1; m += 256) {
+            // R per Y dim (last dim fastest), then f1's repetition digits
+            int32_t r1[kCR], Rraw[kCR];
+#pragma unroll
+            for (int j = 0; j < kCR; ++j) r1[j] = 0;
+            int32_t mm = m;
+#pragma unroll
+            for (int a = kCR - 1; a >= 0; --a) {
+                Rraw[a] = 0;
+                if (a >= cd.ry) continue;
+                const int32_t q = mm / nR[a];
+                const int32_t i = mm - q * nR[a];
+                mm = q;
+                Rraw[a] = R0[a] + i;
+                int32_t R = Rraw[a];
+                if (R >= cd.nRfull[a]) R -= cd.nRfull[a];
+#pragma unroll
+                for (int g = 0; g < kCDig; ++g) {
+                    if (g >= cd.nrd[a]) continue;
+                    const int32_t e = cd.rd_ext[a][g];
+                    const int32_t qq = R / e;
+                    const int32_t dig = R - qq * e;
+                    R = qq;
+                    const int32_t idx = cd.rd_neg[a][g] ? e - 1 - dig : dig;
+#pragma unroll
+                    for (int j = 0; j < kCR; ++j)
+                        if (j == cd.rd_dim[a][g]) r1[j] = idx;
+                }
+            }
+            // f1's reference point in X (o1 + P1 r1 mod sX) and its pattern (Fig. 4)
+            bool in_ok = true;
+            int32_t xb = 0, ref[kCR];
+#pragma unroll
+            for (int a = 0; a < kCR; ++a) {
+                ref[a] = 0;
+                if (a >= cd.rx) continue;
+                int32_t v = cd.o1[a];
+#pragma unroll
+                for (int j = 0; j < kCR; ++j)
+                    if (j < cd.rr1) v += cd.P1[a][j] * r1[j];
+                v -= int32_t(mdiv(uint32_t(v), cd.mX_mul[a], cd.mX_sh[a])) * cd.sX[a];
+                ref[a] = v;
+                in_ok &= v + cd.fmax_in1[a] < cd.sX[a];
+                xb += v * cd.stX[a];
+            }
+            int32_t x[kCP];
+            if (cd.contig1 && in_ok && (xb & 3) == 0 && xb + kCP <= cd.x_elems) {
+#pragma unroll
+                for (int v = 0; v < kCP / 4; ++v) {
+                    if (4 * v >= cd.n_in1) continue;
+                    const int4 q = __ldg(reinterpret_cast<const int4*>(X + xb) + v);
+                    x[4 * v] = q.x;
+                    x[4 * v + 1] = q.y;
+                    x[4 * v + 2] = q.z;
+                    x[4 * v + 3] = q.w;
+                }
+            } else {
+#pragma unroll
+                for (int p = 0; p < kCP; ++p) {
+                    x[p] = 0;
+                    if (p >= cd.n_in1) continue;
+                    int32_t off;
+                    if (in_ok) {
+                        off = xb + cd.lin_in1[p];
+                    } else {
+                        off = 0;
+#pragma unroll
+                        for (int a = 0; a < kCR; ++a) {
+                            if (a >= cd.rx) continue;
+                            int32_t c = ref[a] + cd.f_in1[p][a];   // toroidal pattern element
+                            if (c >= cd.sX[a]) c -= cd.sX[a];
+                            off += c * cd.stX[a];
+                        }
+                    }
+                    x[p] = __ldg(X + off);
+                }
+            }
+            {   // prefix sums: window k = pre[start + len] - pre[start]
+                int32_t acc = 0;
+                my[0] = 0;
+#pragma unroll
+                for (int p = 0; p < kCP; ++p) {
+                    if (p >= cd.n_in1) continue;
+                    acc += x[p];
+                    my[(p + 1) * 256] = acc;
+                }
+            }
+            for (int k = 0; k < cd.nwin1; ++k) {
+                // box position of window k's output: dense index R K + kk relative to the box's first index
+                int32_t off = 0;
+                bool inside = true;
+#pragma unroll
+                for (int a = 0; a < kCR; ++a) {
+                    if (a >= cd.ry) continue;
+                    const int32_t dpos = Rraw[a] * cd.K[a] + cd.kk[k][a] - v0[a];
+                    inside &= dpos >= 0 && dpos < E[a];
+                    off += dpos * bst[a];
+                }
+                if (!inside) continue;
+                const int32_t s0 = cd.start1[k];
+                box[off] = task_c(my[(s0 + cd.len1) * 256] - my[s0 * 256], cd.div1, cd.dv1_mul, cd.dv1_sh);
+            }
+        }
+        __syncthreads();
+        // ---- (2) f2 over the block's repetitions, patterns from the box, outputs to Z
+        const int32_t count = len0 * cd.tail_prod;
+        int32_t zb = cd.zo;
+#pragma unroll
+        for (int j = 0; j < kCR; ++j)
+            if (j < cd.rr2) zb += cd.zP[j] * r2[j];   // outer repetition (inner dims added per repetition)
+        for (int32_t e = threadIdx.x; e < count; e += 256) {
+            uint32_t rem = uint32_t(e);
+            int32_t boff = 0, zoff = zb;
+#pragma unroll
+            for (int d = kCIn - 1; d >= 0; --d) {
+                if (d >= cd.n_inr) continue;
+                int32_t i;
+                if (d == 0) {
+                    i = int32_t(rem);
+                } else {
+                    const uint32_t q = mdiv(rem, cd.in_mul[d], cd.in_sh[d]);
+                    i = int32_t(rem - q * uint32_t(cd.in_len[d]));
+                    rem = q;
+                }
+                int32_t zs = 0;
+#pragma unroll
+                for (int j = 0; j < kCR; ++j)
+                    if (j == cd.in_dim[d]) zs = cd.zP[j];
+                zoff += zs * i;
+#pragma unroll
+                for (int a = 0; a < kCR; ++a) {
+                    if (a >= cd.ry) continue;
+                    int32_t c = 0;
+#pragma unroll
+                    for (int j = 0; j < kCR; ++j)
+                        if (j == cd.in_dim[d]) c = cd.P2[a][j];
+                    if (2 * c > cd.sY[a]) c -= cd.sY[a];
+                    boff += c * i * bst[a];
+                }
+            }
+            {
+                int32_t acc = 0;
+                my[0] = 0;
+#pragma unroll
+                for (int p = 0; p < kCP; ++p) {
+                    if (p >= cd.n_in2) continue;
+                    acc += box[boff + poff[p]];
+                    my[(p + 1) * 256] = acc;
+                }
+            }
+            for (int k = 0; k < cd.nwin2; ++k) {
+                const int32_t s0 = cd.start2[k];
+                Z[zoff + cd.zF[k]] = task_c(my[(s0 + cd.len2) * 256] - my[s0 * 256], cd.div2, cd.dv2_mul, cd.dv2_sh);
+            }
+        }
+        __syncthreads();   // the box is refilled by the next block
+    }
+}
+
+int64_t emod(int64_t a, int64_t m) {
+    const int64_t r = a % m;
+    return r < 0 ? r + m : r;
+}
+
+int64_t signed_rep(int64_t c, int64_t s) {
+    c = emod(c, s);
+    return 2 * c > s ? c - s : c;
+}
+
+void magic_host(uint32_t d, uint32_t* mul, uint32_t* sh) {
+    uint32_t s = 0;
+    while (s < 32 && (uint64_t(1) << s) < uint64_t(d)) ++s;
+    *sh = s;
+    *mul = uint32_t(((uint64_t(1) << 32) * ((uint64_t(1) << s) - uint64_t(d))) / uint64_t(d) + 1);
+}
+
+int64_t prod(const int64_t* s, int n) {
+    int64_t p = 1;
+    for (int k = 0; k < n; ++k) p *= s[k];
+    return p;
+}
+
+// Host plan of the fused chain; false (with a reason) when the chain does not qualify.
+bool plan_chain(const aol_filter_t* f1, const aol_filter_t* f2, ChainDev* cd, int* smem, const char** why) {
+    std::memset(cd, 0, sizeof *cd);
+    const aol_tiler_t& ti = f1->in;
+    const aol_tiler_t& to = f1->out;
+    const aol_tiler_t& t2 = f2->in;
+    const aol_tiler_t& t3 = f2->out;
+    *why = "";
+    if (ti.array_rank > kCR || to.array_rank > kCR || t3.array_rank > kCR || ti.rep_rank > kCR ||
+        t2.rep_rank > kCR) {
+        *why = "ranks above 4";
+        return false;
+    }
+    const int64_t n_in1 = prod(ti.pattern_shape, ti.pattern_rank), n_in2 = prod(t2.pattern_shape, t2.pattern_rank);
+    if (n_in1 > kCP || n_in2 > kCP || f1->n_windows > kCW || f2->n_windows > kCW) {
+        *why = "patterns above 16 elements";
+        return false;
+    }
+    for (const aol_tiler_t* t : {&ti, &to, &t3})
+        if (prod(t->array_shape, t->array_rank) >= (int64_t(1) << 31)) {
+            *why = "arrays of 2^31 elements or more";
+            return false;
+        }
+    // ---- f1 input side (as filter.cu)
+    cd->rx = ti.array_rank;
+    cd->rr1 = ti.rep_rank;
+    int64_t stride = 1;
+    for (int a = ti.array_rank - 1; a >= 0; --a) {
+        cd->sX[a] = int32_t(ti.array_shape[a]);
+        cd->stX[a] = int32_t(stride);
+        stride *= ti.array_shape[a];
+        cd->o1[a] = int32_t(emod(ti.origin[a], ti.array_shape[a]));
+        for (int j = 0; j < ti.rep_rank; ++j) cd->P1[a][j] = int32_t(emod(ti.paving[a][j], ti.array_shape[a]));
+        // o1 + sum P1 r1 must stay below 2^31 before the mod
+        __int128 bound = cd->o1[a];
+        for (int j = 0; j < ti.rep_rank; ++j) bound += __int128(cd->P1[a][j]) * (ti.rep_shape[j] - 1);
+        if (bound >= (__int128(1) << 31)) {
+            *why = "f1 reference points beyond 2^31";
+            return false;
+        }
+        magic_host(uint32_t(cd->sX[a]), &cd->mX_mul[a], &cd->mX_sh[a]);
+    }
+    cd->x_elems = int32_t(stride);
+    cd->n_in1 = int32_t(n_in1);
+    cd->len1 = f1->window_len;
+    cd->nwin1 = f1->n_windows;
+    cd->div1 = f1->divisor;
+    magic_host(uint32_t(f1->divisor < 0 ? -int64_t(f1->divisor) : f1->divisor), &cd->dv1_mul, &cd->dv1_sh);
+    for (int k = 0; k < f1->n_windows; ++k) cd->start1[k] = f1->window_start[k];
+    cd->contig1 = 1;
+    for (int p = 0; p < n_in1; ++p) {
+        int64_t idx[AOL_MAX_RANK] = {0}, q = p;
+        for (int k = ti.pattern_rank - 1; k >= 0; --k) {
+            idx[k] = q % ti.pattern_shape[k];
+            q /= ti.pattern_shape[k];
+        }
+        int64_t lin = 0;
+        for (int a = 0; a < ti.array_rank; ++a) {
+            __int128 v = 0;
+            for (int k = 0; k < ti.pattern_rank; ++k) v += __int128(emod(ti.fitting[a][k], ti.array_shape[a])) * idx[k];
+            cd->f_in1[p][a] = int32_t(v % ti.array_shape[a]);
+            cd->fmax_in1[a] = std::max(cd->fmax_in1[a], cd->f_in1[p][a]);
+            lin += int64_t(cd->f_in1[p][a]) * cd->stX[a];
+        }
+        cd->lin_in1[p] = int32_t(lin);
+        cd->contig1 &= lin == p;
+    }
+    // ---- f1 output side: Y = f1.out.array == f2.in.array; bijective, block-diagonal, window digits low
+    if (to.array_rank != t2.array_rank) {
+        *why = "f1's output array is not f2's input array";
+        return false;
+    }
+    for (int a = 0; a < to.array_rank; ++a)
+        if (to.array_shape[a] != t2.array_shape[a]) {
+            *why = "f1's output array is not f2's input array";
+            return false;
+        }
+    if (prod(to.rep_shape, to.rep_rank) * prod(to.pattern_shape, to.pattern_rank) != prod(to.array_shape, to.array_rank)) {
+        *why = "f1's output tiler does not cover its array exactly";
+        return false;
+    }
+    cd->ry = to.array_rank;
+    // digits: combined dims of f1.out (rep dims j, then pattern dims), each owning one Y dim
+    const int nd = to.rep_rank + to.pattern_rank;
+    int owner[2 * AOL_MAX_RANK];
+    int64_t sstep[2 * AOL_MAX_RANK], ext[2 * AOL_MAX_RANK];
+    for (int d = 0; d < nd; ++d) {
+        ext[d] = d < to.rep_rank ? to.rep_shape[d] : to.pattern_shape[d - to.rep_rank];
+        owner[d] = -1;
+        sstep[d] = 0;
+        if (ext[d] == 1) continue;
+        for (int a = 0; a < to.array_rank; ++a) {
+            const int64_t c = signed_rep(d < to.rep_rank ? to.paving[a][d] : to.fitting[a][d - to.rep_rank],
+                                         to.array_shape[a]);
+            if (c == 0) continue;
+            if (owner[d] >= 0) {
+                *why = "f1's output tiler is not block-diagonal";
+                return false;
+            }
+            owner[d] = a;
+            sstep[d] = c;
+        }
+        if (owner[d] < 0) {
+            *why = "f1's output tiler is not injective";
+            return false;
+        }
+    }
+    // window index k (row-major over f1.out's pattern) -> dense low part per Y dim
+    const int64_t nwin = prod(to.pattern_shape, to.pattern_rank);
+    if (nwin != f1->n_windows) {
+        *why = "f1 windows";
+        return false;
+    }
+    for (int a = 0; a < to.array_rank; ++a) {
+        int ds[2 * AOL_MAX_RANK], n = 0;
+        for (int d = 0; d < nd; ++d)
+            if (ext[d] > 1 && owner[d] == a) ds[n++] = d;
+        std::sort(ds, ds + n, [&](int x, int y) { return std::llabs(sstep[x]) < std::llabs(sstep[y]); });
+        int64_t expect = 1, minraw = 0;
+        bool pattern_part = true;
+        int64_t K = 1;
+        int nrd = 0;
+        for (int q = 0; q < n; ++q) {
+            const int d = ds[q];
+            if (std::llabs(sstep[d]) != expect) {
+                *why = "f1's output tiler is not a dense mixed radix";
+                return false;
+            }
+            expect *= ext[d];
+            if (sstep[d] < 0) minraw += sstep[d] * (ext[d] - 1);
+            if (d >= to.rep_rank) {   // a window (pattern) digit
+                if (!pattern_part) {
+                    *why = "f1's window digits are not the low digits of their Y dim";
+                    return false;
+                }
+                K *= ext[d];
+            } else {
+                pattern_part = false;
+                if (nrd == kCDig) {
+                    *why = "more than 3 repetition digits on one Y dim";
+                    return false;
+                }
+                cd->rd_ext[a][nrd] = int32_t(ext[d]);
+                cd->rd_neg[a][nrd] = sstep[d] < 0;
+                cd->rd_dim[a][nrd] = d;
+                ++nrd;
+            }
+        }
+        if (expect != to.array_shape[a]) {
+            *why = "f1's output tiler does not cover its array exactly";
+            return false;
+        }
+        cd->nrd[a] = nrd;
+        cd->sY[a] = int32_t(to.array_shape[a]);
+        cd->K[a] = int32_t(K);
+        cd->nRfull[a] = int32_t(to.array_shape[a] / K);
+        cd->yo[a] = int32_t(emod(to.origin[a] + minraw, to.array_shape[a]));
+    }
+    for (int a = to.array_rank; a < kCR; ++a) cd->rd_dim[a][0] = -1;
+    for (int a = 0; a < kCR; ++a)
+        for (int g = cd->nrd[a]; g < kCDig; ++g) cd->rd_dim[a][g] = -1;
+    for (int64_t k = 0; k < nwin; ++k) {   // dense low part of window k on each Y dim
+        int64_t idx[AOL_MAX_RANK] = {0}, q = k;
+        for (int p = to.pattern_rank - 1; p >= 0; --p) {
+            idx[p] = q % to.pattern_shape[p];
+            q /= to.pattern_shape[p];
+        }
+        for (int a = 0; a < to.array_rank; ++a) {
+            int64_t v = 0;
+            for (int p = 0; p < to.pattern_rank; ++p) {
+                const int d = to.rep_rank + p;
+                if (owner[d] != a) continue;
+                const int64_t dig = sstep[d] < 0 ? ext[d] - 1 - idx[p] : idx[p];
+                v += std::llabs(sstep[d]) * dig;
+            }
+            cd->kk[k][a] = int32_t(v);
+        }
+    }
+    // ---- f2 input side: blocks of repetitions over a box of Y
+    cd->rr2 = t2.rep_rank;
+    cd->n_in2 = int32_t(n_in2);
+    cd->len2 = f2->window_len;
+    cd->nwin2 = f2->n_windows;
+    cd->div2 = f2->divisor;
+    magic_host(uint32_t(f2->divisor < 0 ? -int64_t(f2->divisor) : f2->divisor), &cd->dv2_mul, &cd->dv2_sh);
+    for (int k = 0; k < f2->n_windows; ++k) cd->start2[k] = f2->window_start[k];
+    for (int a = 0; a < t2.array_rank; ++a) {
+        cd->o2[a] = int32_t(emod(t2.origin[a], t2.array_shape[a]));
+        for (int j = 0; j < t2.rep_rank; ++j) cd->P2[a][j] = int32_t(emod(t2.paving[a][j], t2.array_shape[a]));
+        __int128 bound = cd->o2[a];
+        for (int j = 0; j < t2.rep_rank; ++j) bound += __int128(cd->P2[a][j]) * (t2.rep_shape[j] - 1);
+        if (bound >= (__int128(1) << 31)) {
+            *why = "f2 reference points beyond 2^31";
+            return false;
+        }
+    }
+    int64_t pspan[kCR] = {0};
+    for (int p = 0; p < n_in2; ++p) {
+        int64_t idx[AOL_MAX_RANK] = {0}, q = p;
+        for (int k = t2.pattern_rank - 1; k >= 0; --k) {
+            idx[k] = q % t2.pattern_shape[k];
+            q /= t2.pattern_shape[k];
+        }
+        for (int a = 0; a < t2.array_rank; ++a) {
+            int64_t v = 0;
+            for (int k = 0; k < t2.pattern_rank; ++k) v += signed_rep(t2.fitting[a][k], t2.array_shape[a]) * idx[k];
+            if (std::llabs(v) >= (int64_t(1) << 20)) {
+                *why = "f2 pattern offsets too large";
+                return false;
+            }
+            cd->F2[p][a] = int32_t(v);
+        }
+    }
+    for (int a = 0; a < t2.array_rank; ++a) {
+        int64_t lo = 0, hi = 0;
+        for (int p = 0; p < n_in2; ++p) {
+            lo = std::min<int64_t>(lo, cd->F2[p][a]);
+            hi = std::max<int64_t>(hi, cd->F2[p][a]);
+        }
+        pspan[a] = hi - lo;
+    }
+    // grow the inner repetition block from the innermost rep dim while the box fits; chunk the first that does not
+    const int64_t budget = kChainBox / 4;
+    auto box_vol = [&](int k, int64_t lenk) {
+        int64_t v = 1, last = 1;
+        for (int a = 0; a < t2.array_rank; ++a) {
+            int64_t span = pspan[a];
+            for (int j = k; j < t2.rep_rank; ++j)
+                span += std::llabs(signed_rep(t2.paving[a][j], t2.array_shape[a])) *
+                        ((j == k ? lenk : t2.rep_shape[j]) - 1);
+            v *= span + 1;
+            last = span + 1;
+            if (v > (int64_t(1) << 40)) return int64_t(1) << 40;
+        }
+        return v + v / last;   // + one pad element per row
+    };
+    int k = t2.rep_rank - 1;
+    if (k < 0) {
+        *why = "f2 has no repetition dims";
+        return false;
+    }
+    int64_t lenk = 1;
+    if (box_vol(k, 1) > budget) {
+        *why = "one f2 repetition's pattern box exceeds shared memory";
+        return false;
+    }
+    for (;;) {
+        if (box_vol(k, t2.rep_shape[k]) <= budget) {
+            lenk = t2.rep_shape[k];
+            if (k == 0 || t2.rep_rank - (k - 1) > kCIn || box_vol(k - 1, 1) > budget) break;
+            --k;
+            continue;
+        }
+        int64_t lo = 1, hi = t2.rep_shape[k];
+        while (lo < hi) {
+            const int64_t mid = (lo + hi + 1) / 2;
+            if (box_vol(k, mid) <= budget) lo = mid; else hi = mid - 1;
+        }
+        lenk = lo;
+        break;
+    }
+    cd->n_inr = t2.rep_rank - k;
+    int no = 0;
+    int64_t nblocks = 1;
+    for (int j = 0; j < k; ++j, ++no) {
+        cd->out_dim[no] = j;
+        cd->out_ext[no] = int32_t(t2.rep_shape[j]);
+        magic_host(uint32_t(t2.rep_shape[j]), &cd->out_mul[no], &cd->out_sh[no]);
+        nblocks *= t2.rep_shape[j];
+    }
+    const int64_t nch = (t2.rep_shape[k] + lenk - 1) / lenk;
+    cd->out_dim[no] = k;
+    cd->out_ext[no] = int32_t(nch);
+    magic_host(uint32_t(nch), &cd->out_mul[no], &cd->out_sh[no]);
+    ++no;
+    nblocks *= nch;
+    cd->n_out = no;
+    cd->nblocks = int32_t(nblocks);
+    cd->chunk_ext = int32_t(t2.rep_shape[k]);
+    cd->chunk_len = int32_t(lenk);
+    int64_t tail = 1;
+    for (int d = 0; d < kCIn; ++d) cd->in_dim[d] = -1;
+    for (int d = 0; d < cd->n_inr; ++d) {
+        const int j = k + d;
+        cd->in_dim[d] = j;
+        cd->in_len[d] = int32_t(d == 0 ? lenk : t2.rep_shape[j]);
+        if (d > 0) {
+            magic_host(uint32_t(t2.rep_shape[j]), &cd->in_mul[d], &cd->in_sh[d]);
+            tail *= t2.rep_shape[j];
+        }
+    }
+    cd->tail_prod = int32_t(tail);
+    magic_host(uint32_t(tail), &cd->tail_mul, &cd->tail_sh);
+    // ---- f2 output side: linear (no wrap) Z offsets
+    {
+        int64_t zst[kCR], s = 1;
+        for (int a = t3.array_rank - 1; a >= 0; --a) {
+            zst[a] = s;
+            s *= t3.array_shape[a];
+        }
+        int64_t zo = 0;
+        for (int a = 0; a < t3.array_rank; ++a) {
+            const int64_t o = emod(t3.origin[a], t3.array_shape[a]);
+            __int128 mx = o;
+            for (int j = 0; j < t3.rep_rank; ++j) mx += __int128(emod(t3.paving[a][j], t3.array_shape[a])) * (t3.rep_shape[j] - 1);
+            for (int q = 0; q < t3.pattern_rank; ++q)
+                mx += __int128(emod(t3.fitting[a][q], t3.array_shape[a])) * (t3.pattern_shape[q] - 1);
+            if (mx >= t3.array_shape[a]) {
+                *why = "f2's output tiler wraps";
+                return false;
+            }
+            zo += o * zst[a];
+        }
+        cd->zo = int32_t(zo);
+        for (int j = 0; j < t3.rep_rank; ++j) {
+            int64_t l = 0;
+            for (int a = 0; a < t3.array_rank; ++a) l += emod(t3.paving[a][j], t3.array_shape[a]) * zst[a];
+            cd->zP[j] = int32_t(l);
+        }
+        for (int64_t w = 0; w < f2->n_windows; ++w) {
+            int64_t idx[AOL_MAX_RANK] = {0}, q = w;
+            for (int p = t3.pattern_rank - 1; p >= 0; --p) {
+                idx[p] = q % t3.pattern_shape[p];
+                q /= t3.pattern_shape[p];
+            }
+            int64_t l = 0;
+            for (int a = 0; a < t3.array_rank; ++a)
+                for (int p = 0; p < t3.pattern_rank; ++p) l += emod(t3.fitting[a][p], t3.array_shape[a]) * idx[p] * zst[a];
+            cd->zF[w] = int32_t(l);
+        }
+    }
+    const int64_t box = box_vol(k, lenk);
+    *smem = int((kCP + 1) * 256 * 4 + kCP * 4 + box * 4);
+    return true;
+}
+
+}  // namespace
+}  // namespace aol
+
+using namespace aol;
+
+extern "C" {
+
+aol_status_t aol_filter_chain_apply(const aol_filter_t* f1, const aol_filter_t* f2, const int32_t* d_in, int32_t* d_out,
+                                    void* d_workspace, size_t ws_bytes, cudaStream_t s) {
+    aol_status_t st = aol_filter_validate(f1);
+    if (st != AOL_OK) return st;
+    st = aol_filter_validate(f2);
+    if (st != AOL_OK) return st;
+    if (!d_in || !d_out) return fail(AOL_E_INVALID, "null buffer");
+    if ((reinterpret_cast<uintptr_t>(d_in) | reinterpret_cast<uintptr_t>(d_out)) % 4)
+        return fail(AOL_E_ALIGN, "buffers must be 4-byte aligned");
+    if (f1->out.array_rank != f2->in.array_rank) return fail(AOL_E_SHAPE, "f1's output array is not f2's input array");
+    for (int a = 0; a < f1->out.array_rank; ++a)
+        if (f1->out.array_shape[a] != f2->in.array_shape[a])
+            return fail(AOL_E_SHAPE, "f1's output array is not f2's input array");
+    ChainDev cd;
+    int smem = 0;
+    const char* why = "";
+    const bool fused = std::getenv("AOL_CHAIN_UNFUSED") == nullptr && plan_chain(f1, f2, &cd, &smem, &why);
+    if (!fused) {
+        // two launches through the caller's workspace (the intermediate array)
+        const size_t need = size_t(prod(f1->out.array_shape, f1->out.array_rank)) * 4;
+        if (!d_workspace || ws_bytes < need) {
+            set_error("this chain cannot be fused (%s): it needs a workspace of %zu bytes for the intermediate array",
+                      why, need);
+            return AOL_E_WORKSPACE;
+        }
+        if (reinterpret_cast<uintptr_t>(d_workspace) % 4) return fail(AOL_E_ALIGN, "workspace must be 4-byte aligned");
+        st = aol_filter_apply(f1, d_in, static_cast<int32_t*>(d_workspace), s);
+        if (st != AOL_OK) return st;
+        return aol_filter_apply(f2, static_cast<const int32_t*>(d_workspace), d_out, s);
+    }
+    if (cd.nblocks == 0) return AOL_OK;
+    if (!aligned16(d_in)) cd.contig1 = 0;   // 16-byte pattern loads need an aligned base
+    DeviceInfo dev;
+    st = device_info(&dev);
+    if (st != AOL_OK) return st;
+    st = kernel_smem(reinterpret_cast<const void*>(chain_kernel), smem);
+    if (st != AOL_OK) return st;
+    const int per_sm = std::max(1, kernel_occupancy(reinterpret_cast<const void*>(chain_kernel), 256, smem));
+    const int grid = int(std::max<int64_t>(1, std::min<int64_t>(cd.nblocks, int64_t(dev.num_sms) * per_sm)));
+    st = launch_preflight(reinterpret_cast<const void*>(chain_kernel), 256, smem, "chain_kernel");
+    if (st != AOL_OK) return st;
+    chain_kernel<<<grid, 256, smem, s>>>(cd, d_in, d_out);
+    AOL_LAUNCH_CHECK("chain_kernel");
+    return AOL_OK;
+}
+
+}  // extern "C"

@@ -739,14 +739,38 @@ __device__ __forceinline__ void box_issue_load(const BoxDev& bd, const BoxBlock&
     }
 }
 
+// The VW table entries of a 16-byte output vector (t is a multiple of VW): one 16-byte (or two / four) shared
+// load(s) instead of VW scalar ones (those hit the same bank group from every quarter-warp).
+template <int VW>
+__device__ __forceinline__ void box_tab_vec(const int32_t* tab, int32_t t, int32_t (&o)[VW]) {
+    if constexpr (VW % 4 == 0) {
+#pragma unroll
+        for (int q = 0; q < VW / 4; ++q) {
+            const int4 v = *reinterpret_cast<const int4*>(tab + t + 4 * q);
+            o[4 * q] = v.x;
+            o[4 * q + 1] = v.y;
+            o[4 * q + 2] = v.z;
+            o[4 * q + 3] = v.w;
+        }
+    } else if constexpr (VW == 2) {
+        const int2 v = *reinterpret_cast<const int2*>(tab + t);
+        o[0] = v.x;
+        o[1] = v.y;
+    } else {
+        o[0] = tab[t];
+    }
+}
+
 // smem: [tail_prod] int32 offset table, then one box buffer (FAST scatter) or two (gather: the next block's box
-// loads asynchronously while the current one is written out), each 16-byte aligned.
+// loads asynchronously while the current one is written out), each 16-byte aligned.  A block's geometry is
+// computed once, by thread 0, into shared memory (every thread computing it cost ~20 instructions per element).
 template <int ES, int VW, int MODE>
 __global__ void __launch_bounds__(256) tiler_box_kernel(const __grid_constant__ BoxDev bd, const void* __restrict__ src,
                                                         void* __restrict__ dst, int32_t buf_bytes) {
     using T = typename Elem<ES>::T;
     using VT = typename Vec<ES * VW>::T;
     extern __shared__ __align__(16) uint8_t box_raw[];
+    __shared__ BoxBlock geo[2];
     int32_t* tab = reinterpret_cast<int32_t*>(box_raw);
     uint8_t* bufs = box_raw + ((size_t(bd.tail_prod) * 4 + 15) & ~size_t(15));
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
@@ -755,22 +779,18 @@ __global__ void __launch_bounds__(256) tiler_box_kernel(const __grid_constant__ 
     if (MODE == 0) {
         // software pipeline over this CTA's blocks: box k+1 loads while box k is emitted
         int32_t blk = blockIdx.x;
-        if (blk < bd.nblocks) {
-            BoxBlock b;
-            box_block(bd, blk, b);
-            box_issue_load<ES>(bd, b, src, bufs);
-        }
+        if (threadIdx.x == 0 && blk < bd.nblocks) box_block(bd, blk, geo[0]);
+        __syncthreads();
+        if (blk < bd.nblocks) box_issue_load<ES>(bd, geo[0], src, bufs);
         ptx::cp_async_commit();
         for (int32_t k = 0; blk < bd.nblocks; ++k, blk += gridDim.x) {
             const int32_t nxt = blk + gridDim.x;
-            if (nxt < bd.nblocks) {
-                BoxBlock bn;
-                box_block(bd, nxt, bn);
-                box_issue_load<ES>(bd, bn, src, bufs + ((k + 1) & 1) * buf_bytes);
-            }
+            BoxBlock& gn = geo[(k + 1) & 1];
+            const BoxBlock& b = geo[k & 1];
+            if (threadIdx.x == 0 && nxt < bd.nblocks) box_block(bd, nxt, gn);
+            __syncthreads();
+            if (nxt < bd.nblocks) box_issue_load<ES>(bd, gn, src, bufs + ((k + 1) & 1) * buf_bytes);
             ptx::cp_async_commit();
-            BoxBlock b;
-            box_block(bd, blk, b);
             if (b.len0 != tab_len0) {   // uniform across the CTA; the previous block's reads of tab have finished
                 box_build_table(bd, b, tab);
                 tab_len0 = b.len0;
@@ -779,24 +799,28 @@ __global__ void __launch_bounds__(256) tiler_box_kernel(const __grid_constant__ 
             __syncthreads();
             const T* box = reinterpret_cast<const T*>(bufs + (k & 1) * buf_bytes);
             T* Tg = static_cast<T*>(dst) + b.g0;
-            for (int32_t v = threadIdx.x; v * VW < b.count; v += 256) {
+            const int32_t count = b.count, off0 = b.off0, step0 = b.step[0];
+            for (int32_t v = threadIdx.x; v * VW < count; v += 256) {
                 const uint32_t e = uint32_t(v * VW);
                 const uint32_t i0 = magic_div(e, bd.tail_mul, bd.tail_shift);
                 const int32_t t = int32_t(e - i0 * uint32_t(bd.tail_prod));
-                const int32_t o = b.off0 + b.step[0] * int32_t(i0);
+                const int32_t o = off0 + step0 * int32_t(i0);
+                int32_t to[VW];
+                box_tab_vec<VW>(tab, t, to);
                 union { VT vec; T e[VW]; } pk;
 #pragma unroll
-                for (int j = 0; j < VW; ++j) pk.e[j] = box[o + tab[t + j]];
+                for (int j = 0; j < VW; ++j) pk.e[j] = box[o + to[j]];
                 reinterpret_cast<VT*>(Tg)[v] = pk.vec;
             }
-            __syncthreads();   // this buffer (and tab) may be overwritten from the next iteration on
+            __syncthreads();   // this buffer, its geometry slot and tab may be overwritten from here on
         }
         ptx::cp_async_wait<0>();
     } else {
         T* box = reinterpret_cast<T*>(bufs);
         for (int32_t blk = blockIdx.x; blk < bd.nblocks; blk += gridDim.x) {
-            BoxBlock b;
-            box_block(bd, blk, b);
+            if (threadIdx.x == 0) box_block(bd, blk, geo[0]);
+            __syncthreads();
+            const BoxBlock& b = geo[0];
             const int32_t El = b.E[0], c0 = b.base[0];
             if (b.len0 != tab_len0) {
                 box_build_table(bd, b, tab);
@@ -806,22 +830,25 @@ __global__ void __launch_bounds__(256) tiler_box_kernel(const __grid_constant__ 
             // ---- FAST scatter: the tile block into the box (it covers the box exactly), then the box out;
             // four 16-byte tile loads in flight per thread
             const T* Tg = static_cast<const T*>(src) + b.g0;
+            const int32_t count = b.count, off0 = b.off0, step0 = b.step[0];
             constexpr int kU = 4;
-            for (int32_t v0 = threadIdx.x; v0 * VW < b.count; v0 += 256 * kU) {
+            for (int32_t v0 = threadIdx.x; v0 * VW < count; v0 += 256 * kU) {
                 union { VT vec; T e[VW]; } pk[kU];
 #pragma unroll
                 for (int u = 0; u < kU; ++u)
-                    if ((v0 + 256 * u) * VW < b.count) pk[u].vec = reinterpret_cast<const VT*>(Tg)[v0 + 256 * u];
+                    if ((v0 + 256 * u) * VW < count) pk[u].vec = reinterpret_cast<const VT*>(Tg)[v0 + 256 * u];
 #pragma unroll
                 for (int u = 0; u < kU; ++u) {
                     const int32_t v = v0 + 256 * u;
-                    if (v * VW >= b.count) continue;
+                    if (v * VW >= count) continue;
                     const uint32_t e = uint32_t(v * VW);
                     const uint32_t i0 = magic_div(e, bd.tail_mul, bd.tail_shift);
                     const int32_t t = int32_t(e - i0 * uint32_t(bd.tail_prod));
-                    const int32_t o = b.off0 + b.step[0] * int32_t(i0);
+                    const int32_t o = off0 + step0 * int32_t(i0);
+                    int32_t to[VW];
+                    box_tab_vec<VW>(tab, t, to);
 #pragma unroll
-                    for (int j = 0; j < VW; ++j) box[o + tab[t + j]] = pk[u].e[j];
+                    for (int j = 0; j < VW; ++j) box[o + to[j]] = pk[u].e[j];
                 }
             }
             __syncthreads();
@@ -835,7 +862,7 @@ __global__ void __launch_bounds__(256) tiler_box_kernel(const __grid_constant__ 
                     A[roff + gc] = srow[x];
                 }
             }
-            __syncthreads();
+            __syncthreads();   // the box and geo[0] are rewritten by the next block
         }
     }
 }
