@@ -50,6 +50,8 @@ struct ChainDev {
     int32_t sY[kCR], K[kCR], nRfull[kCR];       // nRfull = sY / K
     int32_t yo[kCR];
     int32_t nrd[kCR], rd_ext[kCR][kCDig], rd_neg[kCR][kCDig], rd_dim[kCR][kCDig];
+    uint32_t rd_mul[kCR][kCDig], rd_sh[kCR][kCDig];
+    int32_t xs[kCR][kCDig][kCR];                 // X reference-point step of digit g of Y dim a, per X dim
     int32_t kk[kCW][kCR];                        // window k's dense low part on each Y dim
     // ---------------- f2: Y -> Z, blocked
     int32_t rr2, n_in2, len2, nwin2, div2;
@@ -66,6 +68,20 @@ struct ChainDev {
     int32_t nblocks;
     // f2's output tiler (linear): Z offset = zo + sum_j zP[j] r_j + zF[k]
     int32_t zo, zP[kCR], zF[kCW];
+    // the same steps per outer / inner repetition dim of the blocking (outer: raw Y steps reduced mod sY, the
+    // chunk dim's per chunk; inner: signed Y steps)
+    int32_t out_y[kCR + 1][kCR], out_z[kCR + 1];
+    int32_t in_y[kCIn][kCR], in_z[kCIn];
+};
+
+// Per-block quantities, computed once by thread 0 into shared memory.
+struct ChainBlk {
+    int32_t E[kCR], base[kCR], bst[kCR], lo[kCR];   // Y box: extents, corner (mod sY), smem strides, corner offset
+    int32_t v0[kCR], R0[kCR], nR[kCR];               // f1 repetitions covering the box: R0 .. R0 + nR - 1 per Y dim
+    uint32_t nR_mul[kCR], nR_sh[kCR];
+    int32_t nrep1, len0, count, zb;
+    int32_t bstep[kCIn];                             // box offset per unit of inner repetition dim d
+    int32_t poff[kCP];                               // box offset of f2 pattern element p (relative)
 };
 
 __device__ __forceinline__ uint32_t mdiv(uint32_t n, uint32_t mul, uint32_t sh) { return (__umulhi(n, mul) + n) >> sh; }
@@ -77,153 +93,122 @@ __device__ __forceinline__ int32_t task_c(int32_t S, int32_t d, uint32_t mul, ui
     return q * (1 + d) - S;
 }
 
+__device__ __forceinline__ void magic_dev(uint32_t d, uint32_t& mul, uint32_t& sh) {
+    uint32_t s = 0;
+    while (s < 32 && (1ull << s) < d) ++s;
+    sh = s;
+    mul = uint32_t(((1ull << 32) * ((1ull << s) - uint64_t(d))) / d + 1);
+}
+
+__device__ void chain_block(const ChainDev& cd, int32_t blk, ChainBlk& g, int RY) {
+    int64_t raw[kCR];
+    for (int a = 0; a < kCR; ++a) raw[a] = cd.o2[a];
+    int32_t zb = cd.zo;
+    uint32_t n = uint32_t(blk);
+    int32_t ck = 0;
+    for (int d = cd.n_out - 1; d >= 0; --d) {
+        const uint32_t q = mdiv(n, cd.out_mul[d], cd.out_sh[d]);
+        const int32_t i = int32_t(n - q * uint32_t(cd.out_ext[d]));
+        n = q;
+        if (d == cd.n_out - 1) ck = i;
+        for (int a = 0; a < RY; ++a) raw[a] += int64_t(cd.out_y[d][a]) * i;
+        zb += cd.out_z[d] * i;
+    }
+    g.len0 = min(cd.chunk_len, cd.chunk_ext - ck * cd.chunk_len);
+    g.count = g.len0 * cd.tail_prod;
+    g.zb = zb;
+    int32_t st = 1;
+    g.nrep1 = 1;
+    for (int a = RY - 1; a >= 0; --a) {
+        int32_t l = 0, h = 0;
+        for (int d = 0; d < cd.n_inr; ++d) {
+            const int32_t c = cd.in_y[d][a], ln = (d == 0 ? g.len0 : cd.in_len[d]) - 1;
+            if (c < 0) l += c * ln; else h += c * ln;
+        }
+        int32_t pl = 0, ph = 0;
+        for (int p = 0; p < cd.n_in2; ++p) {
+            pl = min(pl, cd.F2[p][a]);
+            ph = max(ph, cd.F2[p][a]);
+        }
+        l += pl;
+        h += ph;
+        g.E[a] = h - l + 1;
+        int32_t v = int32_t((raw[a] + l) % cd.sY[a]);
+        g.base[a] = v < 0 ? v + cd.sY[a] : v;
+        g.lo[a] = l;
+        g.bst[a] = st;
+        st *= (a == RY - 1) ? g.E[a] + ((g.E[a] & 31) == 0 ? 1 : 0) : g.E[a];
+        // f1 repetitions covering the dense index range [v0, v0 + E) of this Y dim
+        v = g.base[a] - cd.yo[a];
+        if (v < 0) v += cd.sY[a];
+        g.v0[a] = v;
+        g.R0[a] = v / cd.K[a];
+        g.nR[a] = (v + g.E[a] - 1) / cd.K[a] - g.R0[a] + 1;
+        magic_dev(uint32_t(g.nR[a]), g.nR_mul[a], g.nR_sh[a]);
+        g.nrep1 *= g.nR[a];
+    }
+    for (int d = 0; d < cd.n_inr; ++d) {
+        int32_t o = 0;
+        for (int a = 0; a < RY; ++a) o += cd.in_y[d][a] * g.bst[a];
+        g.bstep[d] = o;
+    }
+    for (int p = 0; p < cd.n_in2; ++p) {
+        int32_t o = 0;
+        for (int a = 0; a < RY; ++a) o += (cd.F2[p][a] - g.lo[a]) * g.bst[a];
+        g.poff[p] = o;
+    }
+}
+
+template <int RX, int RY>
 __global__ void __launch_bounds__(256) chain_kernel(const __grid_constant__ ChainDev cd, const int32_t* __restrict__ X,
                                                     int32_t* __restrict__ Z) {
     extern __shared__ __align__(16) int32_t sm[];
+    __shared__ ChainBlk g;
     int32_t* pre = sm;                          // [kCP + 1][256] per-thread prefix sums
-    int32_t* poff = pre + (kCP + 1) * 256;      // [kCP] f2 pattern offsets in the box
-    int32_t* box = poff + kCP;
+    int32_t* box = pre + (kCP + 1) * 256;
     int32_t* my = pre + threadIdx.x;
     for (int32_t blk = blockIdx.x; blk < cd.nblocks; blk += gridDim.x) {
-        // ---- block geometry: f2 outer repetition index, box over Y
-        int32_t r2[kCR];
-#pragma unroll
-        for (int j = 0; j < kCR; ++j) r2[j] = 0;
-        uint32_t n = uint32_t(blk);
-        int32_t ck = 0;
-        for (int d = cd.n_out - 1; d >= 0; --d) {
-            const uint32_t q = mdiv(n, cd.out_mul[d], cd.out_sh[d]);
-            const int32_t i = int32_t(n - q * uint32_t(cd.out_ext[d]));
-            n = q;
-            if (d == cd.n_out - 1) ck = i;
-            else {
-#pragma unroll
-                for (int j = 0; j < kCR; ++j)
-                    if (j == cd.out_dim[d]) r2[j] = i;
-            }
-        }
-        const int32_t len0 = min(cd.chunk_len, cd.chunk_ext - ck * cd.chunk_len);
-#pragma unroll
-        for (int j = 0; j < kCR; ++j)
-            if (j == cd.in_dim[0]) r2[j] = ck * cd.chunk_len;
-        // box extents / corner per Y dim (raw = o2 + P2 r2 + [lo, hi] over inner reps and pattern)
-        int32_t E[kCR], base[kCR], lo[kCR], bst[kCR];
-        int32_t rows = 1, pitch = 1, st = 1;
-#pragma unroll
-        for (int a = kCR - 1; a >= 0; --a) {
-            E[a] = 1;
-            base[a] = 0;
-            lo[a] = 0;
-            bst[a] = 0;
-            if (a >= cd.ry) continue;
-            int64_t raw = cd.o2[a];
-#pragma unroll
-            for (int j = 0; j < kCR; ++j)
-                if (j < cd.rr2) raw += int64_t(cd.P2[a][j]) * r2[j];
-            int32_t l = 0, h = 0;
-#pragma unroll
-            for (int d = 0; d < kCIn; ++d) {
-                if (d >= cd.n_inr) continue;
-                int32_t c = 0;
-#pragma unroll
-                for (int j = 0; j < kCR; ++j)
-                    if (j == cd.in_dim[d]) c = cd.P2[a][j];
-                if (2 * c > cd.sY[a]) c -= cd.sY[a];   // signed step
-                const int32_t ln = (d == 0 ? len0 : cd.in_len[d]) - 1;
-                if (c < 0) l += c * ln; else h += c * ln;
-            }
-            int32_t pl = 0, ph = 0;
-            for (int p = 0; p < cd.n_in2; ++p) {
-                pl = min(pl, cd.F2[p][a]);
-                ph = max(ph, cd.F2[p][a]);
-            }
-            l += pl;
-            h += ph;
-            E[a] = h - l + 1;
-            const int32_t v = int32_t((raw + l) % cd.sY[a]);
-            base[a] = v < 0 ? v + cd.sY[a] : v;
-            lo[a] = l;
-            bst[a] = st;
-            if (a == cd.ry - 1) {
-                pitch = E[a] + ((E[a] & 31) == 0 ? 1 : 0);
-                st = pitch;
-            } else {
-                st *= E[a];
-                rows *= E[a];
-            }
-        }
-        if (threadIdx.x < cd.n_in2) {
-            int32_t o = 0;
-#pragma unroll
-            for (int a = 0; a < kCR; ++a)
-                if (a < cd.ry) o += (cd.F2[threadIdx.x][a] - lo[a]) * bst[a];   // box offset of element p at r2
-            poff[threadIdx.x] = o;
-        }
-        // ---- (1) fill the box with f1: repetitions covering the box, a contiguous range of R per Y dim
-        int32_t R0[kCR], nR[kCR], v0[kCR];
-        int32_t nrep1 = 1;
-#pragma unroll
-        for (int a = 0; a < kCR; ++a) {
-            R0[a] = 0;
-            nR[a] = 1;
-            v0[a] = 0;
-            if (a >= cd.ry) continue;
-            int32_t v = base[a] - cd.yo[a];
-            if (v < 0) v += cd.sY[a];
-            v0[a] = v;
-            R0[a] = v / cd.K[a];
-            nR[a] = min((v + E[a] - 1) / cd.K[a] - R0[a] + 1, cd.nRfull[a] + 1);
-            nrep1 *= nR[a];
-        }
+        if (threadIdx.x == 0) chain_block(cd, blk, g, RY);
+        __syncthreads();
+        // ---- (1) fill the box with f1 over the repetitions whose outputs land in it
+        const int32_t nrep1 = g.nrep1;
         for (int32_t m = threadIdx.x; m < nrep1; m += 256) {
-            // R per Y dim (last dim fastest), then f1's repetition digits
-            int32_t r1[kCR], Rraw[kCR];
+            int32_t ref[RX], Rraw[RY];
 #pragma unroll
-            for (int j = 0; j < kCR; ++j) r1[j] = 0;
-            int32_t mm = m;
+            for (int ax = 0; ax < RX; ++ax) ref[ax] = cd.o1[ax];
+            uint32_t mm = uint32_t(m);
 #pragma unroll
-            for (int a = kCR - 1; a >= 0; --a) {
-                Rraw[a] = 0;
-                if (a >= cd.ry) continue;
-                const int32_t q = mm / nR[a];
-                const int32_t i = mm - q * nR[a];
+            for (int a = RY - 1; a >= 0; --a) {
+                const uint32_t q = mdiv(mm, g.nR_mul[a], g.nR_sh[a]);
+                const int32_t i = int32_t(mm - q * uint32_t(g.nR[a]));
                 mm = q;
-                Rraw[a] = R0[a] + i;
-                int32_t R = Rraw[a];
-                if (R >= cd.nRfull[a]) R -= cd.nRfull[a];
+                Rraw[a] = g.R0[a] + i;
+                uint32_t R = uint32_t(Rraw[a] >= cd.nRfull[a] ? Rraw[a] - cd.nRfull[a] : Rraw[a]);
+                while (R >= uint32_t(cd.nRfull[a])) R -= uint32_t(cd.nRfull[a]);
 #pragma unroll
-                for (int g = 0; g < kCDig; ++g) {
-                    if (g >= cd.nrd[a]) continue;
-                    const int32_t e = cd.rd_ext[a][g];
-                    const int32_t qq = R / e;
-                    const int32_t dig = R - qq * e;
-                    R = qq;
-                    const int32_t idx = cd.rd_neg[a][g] ? e - 1 - dig : dig;
+                for (int gg = 0; gg < kCDig; ++gg) {
+                    if (gg >= cd.nrd[a]) continue;
+                    const uint32_t q2 = mdiv(R, cd.rd_mul[a][gg], cd.rd_sh[a][gg]);
+                    const int32_t dig = int32_t(R - q2 * uint32_t(cd.rd_ext[a][gg]));
+                    R = q2;
+                    const int32_t idx = cd.rd_neg[a][gg] ? cd.rd_ext[a][gg] - 1 - dig : dig;
 #pragma unroll
-                    for (int j = 0; j < kCR; ++j)
-                        if (j == cd.rd_dim[a][g]) r1[j] = idx;
+                    for (int ax = 0; ax < RX; ++ax) ref[ax] += cd.xs[a][gg][ax] * idx;
                 }
             }
-            // f1's reference point in X (o1 + P1 r1 mod sX) and its pattern (Fig. 4)
             bool in_ok = true;
-            int32_t xb = 0, ref[kCR];
+            int32_t xb = 0;
 #pragma unroll
-            for (int a = 0; a < kCR; ++a) {
-                ref[a] = 0;
-                if (a >= cd.rx) continue;
-                int32_t v = cd.o1[a];
-#pragma unroll
-                for (int j = 0; j < kCR; ++j)
-                    if (j < cd.rr1) v += cd.P1[a][j] * r1[j];
-                v -= int32_t(mdiv(uint32_t(v), cd.mX_mul[a], cd.mX_sh[a])) * cd.sX[a];
-                ref[a] = v;
-                in_ok &= v + cd.fmax_in1[a] < cd.sX[a];
-                xb += v * cd.stX[a];
+            for (int ax = 0; ax < RX; ++ax) {
+                ref[ax] -= int32_t(mdiv(uint32_t(ref[ax]), cd.mX_mul[ax], cd.mX_sh[ax])) * cd.sX[ax];
+                in_ok &= ref[ax] + cd.fmax_in1[ax] < cd.sX[ax];
+                xb += ref[ax] * cd.stX[ax];
             }
             int32_t x[kCP];
             if (cd.contig1 && in_ok && (xb & 3) == 0 && xb + kCP <= cd.x_elems) {
 #pragma unroll
                 for (int v = 0; v < kCP / 4; ++v) {
+                    x[4 * v] = x[4 * v + 1] = x[4 * v + 2] = x[4 * v + 3] = 0;
                     if (4 * v >= cd.n_in1) continue;
                     const int4 q = __ldg(reinterpret_cast<const int4*>(X + xb) + v);
                     x[4 * v] = q.x;
@@ -242,11 +227,10 @@ __global__ void __launch_bounds__(256) chain_kernel(const __grid_constant__ Chai
                     } else {
                         off = 0;
 #pragma unroll
-                        for (int a = 0; a < kCR; ++a) {
-                            if (a >= cd.rx) continue;
-                            int32_t c = ref[a] + cd.f_in1[p][a];   // toroidal pattern element
-                            if (c >= cd.sX[a]) c -= cd.sX[a];
-                            off += c * cd.stX[a];
+                        for (int ax = 0; ax < RX; ++ax) {
+                            int32_t c = ref[ax] + cd.f_in1[p][ax];   // toroidal pattern element
+                            if (c >= cd.sX[ax]) c -= cd.sX[ax];
+                            off += c * cd.stX[ax];
                         }
                     }
                     x[p] = __ldg(X + off);
@@ -262,16 +246,17 @@ __global__ void __launch_bounds__(256) chain_kernel(const __grid_constant__ Chai
                     my[(p + 1) * 256] = acc;
                 }
             }
-            for (int k = 0; k < cd.nwin1; ++k) {
-                // box position of window k's output: dense index R K + kk relative to the box's first index
-                int32_t off = 0;
-                bool inside = true;
+            int32_t dbase = 0;   // box offset of the repetition's dense point R K (window offsets added below)
 #pragma unroll
-                for (int a = 0; a < kCR; ++a) {
-                    if (a >= cd.ry) continue;
-                    const int32_t dpos = Rraw[a] * cd.K[a] + cd.kk[k][a] - v0[a];
-                    inside &= dpos >= 0 && dpos < E[a];
-                    off += dpos * bst[a];
+            for (int a = 0; a < RY; ++a) dbase += (Rraw[a] * cd.K[a] - g.v0[a]) * g.bst[a];
+            for (int k = 0; k < cd.nwin1; ++k) {
+                bool inside = true;
+                int32_t off = dbase;
+#pragma unroll
+                for (int a = 0; a < RY; ++a) {
+                    const int32_t dpos = Rraw[a] * cd.K[a] + cd.kk[k][a] - g.v0[a];
+                    inside &= dpos >= 0 && dpos < g.E[a];
+                    off += cd.kk[k][a] * g.bst[a];
                 }
                 if (!inside) continue;
                 const int32_t s0 = cd.start1[k];
@@ -280,48 +265,28 @@ __global__ void __launch_bounds__(256) chain_kernel(const __grid_constant__ Chai
         }
         __syncthreads();
         // ---- (2) f2 over the block's repetitions, patterns from the box, outputs to Z
-        const int32_t count = len0 * cd.tail_prod;
-        int32_t zb = cd.zo;
-#pragma unroll
-        for (int j = 0; j < kCR; ++j)
-            if (j < cd.rr2) zb += cd.zP[j] * r2[j];   // outer repetition (inner dims added per repetition)
+        const int32_t count = g.count, zb = g.zb;
         for (int32_t e = threadIdx.x; e < count; e += 256) {
             uint32_t rem = uint32_t(e);
             int32_t boff = 0, zoff = zb;
 #pragma unroll
-            for (int d = kCIn - 1; d >= 0; --d) {
+            for (int d = kCIn - 1; d >= 1; --d) {
                 if (d >= cd.n_inr) continue;
-                int32_t i;
-                if (d == 0) {
-                    i = int32_t(rem);
-                } else {
-                    const uint32_t q = mdiv(rem, cd.in_mul[d], cd.in_sh[d]);
-                    i = int32_t(rem - q * uint32_t(cd.in_len[d]));
-                    rem = q;
-                }
-                int32_t zs = 0;
-#pragma unroll
-                for (int j = 0; j < kCR; ++j)
-                    if (j == cd.in_dim[d]) zs = cd.zP[j];
-                zoff += zs * i;
-#pragma unroll
-                for (int a = 0; a < kCR; ++a) {
-                    if (a >= cd.ry) continue;
-                    int32_t c = 0;
-#pragma unroll
-                    for (int j = 0; j < kCR; ++j)
-                        if (j == cd.in_dim[d]) c = cd.P2[a][j];
-                    if (2 * c > cd.sY[a]) c -= cd.sY[a];
-                    boff += c * i * bst[a];
-                }
+                const uint32_t q = mdiv(rem, cd.in_mul[d], cd.in_sh[d]);
+                const int32_t i = int32_t(rem - q * uint32_t(cd.in_len[d]));
+                rem = q;
+                boff += g.bstep[d] * i;
+                zoff += cd.in_z[d] * i;
             }
+            boff += g.bstep[0] * int32_t(rem);
+            zoff += cd.in_z[0] * int32_t(rem);
             {
                 int32_t acc = 0;
                 my[0] = 0;
 #pragma unroll
                 for (int p = 0; p < kCP; ++p) {
                     if (p >= cd.n_in2) continue;
-                    acc += box[boff + poff[p]];
+                    acc += box[boff + g.poff[p]];
                     my[(p + 1) * 256] = acc;
                 }
             }
@@ -330,8 +295,19 @@ __global__ void __launch_bounds__(256) chain_kernel(const __grid_constant__ Chai
                 Z[zoff + cd.zF[k]] = task_c(my[(s0 + cd.len2) * 256] - my[s0 * 256], cd.div2, cd.dv2_mul, cd.dv2_sh);
             }
         }
-        __syncthreads();   // the box is refilled by the next block
+        __syncthreads();   // the box and g are rewritten by the next block
     }
+}
+
+using ChainFn = void (*)(const ChainDev, const int32_t*, int32_t*);
+
+ChainFn chain_kernel_for(int rx, int ry) {
+    static const ChainFn tab[4][4] = {
+        {chain_kernel<1, 1>, chain_kernel<1, 2>, chain_kernel<1, 3>, chain_kernel<1, 4>},
+        {chain_kernel<2, 1>, chain_kernel<2, 2>, chain_kernel<2, 3>, chain_kernel<2, 4>},
+        {chain_kernel<3, 1>, chain_kernel<3, 2>, chain_kernel<3, 3>, chain_kernel<3, 4>},
+        {chain_kernel<4, 1>, chain_kernel<4, 2>, chain_kernel<4, 3>, chain_kernel<4, 4>}};
+    return tab[rx - 1][ry - 1];
 }
 
 int64_t emod(int64_t a, int64_t m) {
@@ -502,6 +478,8 @@ bool plan_chain(const aol_filter_t* f1, const aol_filter_t* f2, ChainDev* cd, in
                 cd->rd_ext[a][nrd] = int32_t(ext[d]);
                 cd->rd_neg[a][nrd] = sstep[d] < 0;
                 cd->rd_dim[a][nrd] = d;
+                magic_host(uint32_t(ext[d]), &cd->rd_mul[a][nrd], &cd->rd_sh[a][nrd]);
+                for (int ax = 0; ax < ti.array_rank; ++ax) cd->xs[a][nrd][ax] = cd->P1[ax][d];
                 ++nrd;
             }
         }
@@ -688,8 +666,20 @@ bool plan_chain(const aol_filter_t* f1, const aol_filter_t* f2, ChainDev* cd, in
             cd->zF[w] = int32_t(l);
         }
     }
+    // per blocking dim: Y raw steps (outer: reduced mod sY, the chunk dim per chunk; inner: signed) and Z steps
+    for (int d = 0; d < cd->n_out; ++d) {
+        const int j = cd->out_dim[d];
+        const int64_t mult = d == cd->n_out - 1 ? lenk : 1;
+        for (int a = 0; a < t2.array_rank; ++a) cd->out_y[d][a] = int32_t(emod(int64_t(cd->P2[a][j]) * mult, t2.array_shape[a]));
+        cd->out_z[d] = int32_t(int64_t(cd->zP[j]) * mult);
+    }
+    for (int d = 0; d < cd->n_inr; ++d) {
+        const int j = cd->in_dim[d];
+        for (int a = 0; a < t2.array_rank; ++a) cd->in_y[d][a] = int32_t(signed_rep(cd->P2[a][j], t2.array_shape[a]));
+        cd->in_z[d] = cd->zP[j];
+    }
     const int64_t box = box_vol(k, lenk);
-    *smem = int((kCP + 1) * 256 * 4 + kCP * 4 + box * 4);
+    *smem = int((kCP + 1) * 256 * 4 + box * 4);
     return true;
 }
 
@@ -735,13 +725,14 @@ aol_status_t aol_filter_chain_apply(const aol_filter_t* f1, const aol_filter_t* 
     DeviceInfo dev;
     st = device_info(&dev);
     if (st != AOL_OK) return st;
-    st = kernel_smem(reinterpret_cast<const void*>(chain_kernel), smem);
+    const ChainFn kern = chain_kernel_for(cd.rx, cd.ry);
+    st = kernel_smem(reinterpret_cast<const void*>(kern), smem);
     if (st != AOL_OK) return st;
-    const int per_sm = std::max(1, kernel_occupancy(reinterpret_cast<const void*>(chain_kernel), 256, smem));
+    const int per_sm = std::max(1, kernel_occupancy(reinterpret_cast<const void*>(kern), 256, smem));
     const int grid = int(std::max<int64_t>(1, std::min<int64_t>(cd.nblocks, int64_t(dev.num_sms) * per_sm)));
-    st = launch_preflight(reinterpret_cast<const void*>(chain_kernel), 256, smem, "chain_kernel");
+    st = launch_preflight(reinterpret_cast<const void*>(kern), 256, smem, "chain_kernel");
     if (st != AOL_OK) return st;
-    chain_kernel<<<grid, 256, smem, s>>>(cd, d_in, d_out);
+    kern<<<grid, 256, smem, s>>>(cd, d_in, d_out);
     AOL_LAUNCH_CHECK("chain_kernel");
     return AOL_OK;
 }
