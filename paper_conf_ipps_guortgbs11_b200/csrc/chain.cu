@@ -53,6 +53,7 @@ struct ChainDev {
     uint32_t rd_mul[kCR][kCDig], rd_sh[kCR][kCDig];
     int32_t xs[kCR][kCDig][kCR];                 // X reference-point step of digit g of Y dim a, per X dim
     int32_t kk[kCW][kCR];                        // window k's dense low part on each Y dim
+    int32_t kkmin[kCR], kkmax[kCR];              // their range per Y dim
     // ---------------- f2: Y -> Z, blocked
     int32_t rr2, n_in2, len2, nwin2, div2;
     uint32_t dv2_mul, dv2_sh;
@@ -82,6 +83,8 @@ struct ChainBlk {
     int32_t nrep1, len0, count, zb;
     int32_t bstep[kCIn];                             // box offset per unit of inner repetition dim d
     int32_t poff[kCP];                               // box offset of f2 pattern element p (relative)
+    int32_t kkoff[kCW];                              // box offset of f1 window k relative to its repetition
+    int32_t nrow1;                                   // f1: rows of repetitions (all Y dims but the last)
 };
 
 __device__ __forceinline__ uint32_t mdiv(uint32_t n, uint32_t mul, uint32_t sh) { return (__umulhi(n, mul) + n) >> sh; }
@@ -157,9 +160,111 @@ __device__ void chain_block(const ChainDev& cd, int32_t blk, ChainBlk& g, int RY
         for (int a = 0; a < RY; ++a) o += (cd.F2[p][a] - g.lo[a]) * g.bst[a];
         g.poff[p] = o;
     }
+    for (int k = 0; k < cd.nwin1; ++k) {
+        int32_t o = 0;
+        for (int a = 0; a < RY; ++a) o += cd.kk[k][a] * g.bst[a];
+        g.kkoff[k] = o;
+    }
+    g.nrow1 = g.nrep1 / g.nR[RY - 1];
 }
 
-template <int RX, int RY>
+// f1's repetition with dense coordinates Rraw (per Y dim) at X reference point ref: gather its pattern, window
+// sums, task, and store the outputs that fall inside the box (all of them when `all_in`).
+template <int RX, int RY, int NP1>
+__device__ __forceinline__ void chain_f1_rep(const ChainDev& cd, const ChainBlk& g, const int32_t* __restrict__ X,
+                                             int32_t* box, int32_t* my, int32_t (&ref)[RX], const int32_t (&Rraw)[RY]) {
+    bool in_ok = true;
+    int32_t xb = 0;
+#pragma unroll
+    for (int ax = 0; ax < RX; ++ax) {
+        ref[ax] -= int32_t(mdiv(uint32_t(ref[ax]), cd.mX_mul[ax], cd.mX_sh[ax])) * cd.sX[ax];
+        in_ok &= ref[ax] + cd.fmax_in1[ax] < cd.sX[ax];
+        xb += ref[ax] * cd.stX[ax];
+    }
+    int32_t x[NP1];
+    if (cd.contig1 && in_ok && (xb & 3) == 0 && xb + NP1 <= cd.x_elems) {
+#pragma unroll
+        for (int v = 0; v < NP1 / 4; ++v) {
+            const int4 q = __ldg(reinterpret_cast<const int4*>(X + xb) + v);
+            x[4 * v] = q.x;
+            x[4 * v + 1] = q.y;
+            x[4 * v + 2] = q.z;
+            x[4 * v + 3] = q.w;
+        }
+    } else {
+#pragma unroll
+        for (int p = 0; p < NP1; ++p) {
+            x[p] = 0;
+            if (p >= cd.n_in1) continue;
+            int32_t off;
+            if (in_ok) {
+                off = xb + cd.lin_in1[p];
+            } else {
+                off = 0;
+#pragma unroll
+                for (int ax = 0; ax < RX; ++ax) {
+                    int32_t c = ref[ax] + cd.f_in1[p][ax];   // toroidal pattern element
+                    if (c >= cd.sX[ax]) c -= cd.sX[ax];
+                    off += c * cd.stX[ax];
+                }
+            }
+            x[p] = __ldg(X + off);
+        }
+    }
+    {   // prefix sums (elements past the pattern are never read by a window)
+        int32_t acc = 0;
+        my[0] = 0;
+#pragma unroll
+        for (int p = 0; p < NP1; ++p) {
+            acc += x[p];
+            my[(p + 1) * 256] = acc;
+        }
+    }
+    int32_t dbase = 0;
+    bool all_in = true;
+#pragma unroll
+    for (int a = 0; a < RY; ++a) {
+        const int32_t d0 = Rraw[a] * cd.K[a] - g.v0[a];
+        dbase += d0 * g.bst[a];
+        all_in &= d0 + cd.kkmin[a] >= 0 && d0 + cd.kkmax[a] < g.E[a];
+    }
+    for (int k = 0; k < cd.nwin1; ++k) {
+        if (!all_in) {
+            bool inside = true;
+#pragma unroll
+            for (int a = 0; a < RY; ++a) {
+                const int32_t dpos = Rraw[a] * cd.K[a] + cd.kk[k][a] - g.v0[a];
+                inside &= dpos >= 0 && dpos < g.E[a];
+            }
+            if (!inside) continue;
+        }
+        const int32_t s0 = cd.start1[k];
+        box[dbase + g.kkoff[k]] = task_c(my[(s0 + cd.len1) * 256] - my[s0 * 256], cd.div1, cd.dv1_mul, cd.dv1_sh);
+    }
+}
+
+// The f1 reference-point contribution of Y dim a's dense repetition coordinate Rraw (digits of R mod nRfull).
+template <int RX>
+__device__ __forceinline__ void chain_digits(const ChainDev& cd, int a, int32_t Rraw, int32_t (&ref)[RX]) {
+    uint32_t R = uint32_t(Rraw);
+    while (R >= uint32_t(cd.nRfull[a])) R -= uint32_t(cd.nRfull[a]);
+#pragma unroll
+    for (int gg = 0; gg < kCDig; ++gg) {
+        if (gg >= cd.nrd[a]) continue;
+        uint32_t q2 = 0;
+        int32_t dig = int32_t(R);
+        if (gg + 1 < cd.nrd[a]) {   // the last digit is the remaining quotient itself
+            q2 = mdiv(R, cd.rd_mul[a][gg], cd.rd_sh[a][gg]);
+            dig = int32_t(R - q2 * uint32_t(cd.rd_ext[a][gg]));
+        }
+        R = q2;
+        const int32_t idx = cd.rd_neg[a][gg] ? cd.rd_ext[a][gg] - 1 - dig : dig;
+#pragma unroll
+        for (int ax = 0; ax < RX; ++ax) ref[ax] += cd.xs[a][gg][ax] * idx;
+    }
+}
+
+template <int RX, int RY, int NP1>
 __global__ void __launch_bounds__(256) chain_kernel(const __grid_constant__ ChainDev cd, const int32_t* __restrict__ X,
                                                     int32_t* __restrict__ Z) {
     extern __shared__ __align__(16) int32_t sm[];
@@ -167,132 +272,70 @@ __global__ void __launch_bounds__(256) chain_kernel(const __grid_constant__ Chai
     int32_t* pre = sm;                          // [kCP + 1][256] per-thread prefix sums
     int32_t* box = pre + (kCP + 1) * 256;
     int32_t* my = pre + threadIdx.x;
+    const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
     for (int32_t blk = blockIdx.x; blk < cd.nblocks; blk += gridDim.x) {
         if (threadIdx.x == 0) chain_block(cd, blk, g, RY);
         __syncthreads();
-        // ---- (1) fill the box with f1 over the repetitions whose outputs land in it
-        const int32_t nrep1 = g.nrep1;
-        for (int32_t m = threadIdx.x; m < nrep1; m += 256) {
-            int32_t ref[RX], Rraw[RY];
+        // ---- (1) fill the box with f1: a warp per row of covering repetitions (all Y dims but the last fixed),
+        // lanes along the last Y dim's repetition range (coalesced X patterns)
+        const int32_t nrow1 = g.nrow1, nlast = g.nR[RY - 1];
+        for (int32_t row = warp; row < nrow1; row += 8) {
+            int32_t rref[RX], Rraw[RY];
 #pragma unroll
-            for (int ax = 0; ax < RX; ++ax) ref[ax] = cd.o1[ax];
-            uint32_t mm = uint32_t(m);
+            for (int ax = 0; ax < RX; ++ax) rref[ax] = cd.o1[ax];
+            uint32_t mm = uint32_t(row);
 #pragma unroll
-            for (int a = RY - 1; a >= 0; --a) {
+            for (int a = RY - 2; a >= 0; --a) {
                 const uint32_t q = mdiv(mm, g.nR_mul[a], g.nR_sh[a]);
                 const int32_t i = int32_t(mm - q * uint32_t(g.nR[a]));
                 mm = q;
                 Rraw[a] = g.R0[a] + i;
-                uint32_t R = uint32_t(Rraw[a] >= cd.nRfull[a] ? Rraw[a] - cd.nRfull[a] : Rraw[a]);
-                while (R >= uint32_t(cd.nRfull[a])) R -= uint32_t(cd.nRfull[a]);
-#pragma unroll
-                for (int gg = 0; gg < kCDig; ++gg) {
-                    if (gg >= cd.nrd[a]) continue;
-                    const uint32_t q2 = mdiv(R, cd.rd_mul[a][gg], cd.rd_sh[a][gg]);
-                    const int32_t dig = int32_t(R - q2 * uint32_t(cd.rd_ext[a][gg]));
-                    R = q2;
-                    const int32_t idx = cd.rd_neg[a][gg] ? cd.rd_ext[a][gg] - 1 - dig : dig;
-#pragma unroll
-                    for (int ax = 0; ax < RX; ++ax) ref[ax] += cd.xs[a][gg][ax] * idx;
-                }
+                chain_digits<RX>(cd, a, Rraw[a], rref);
             }
-            bool in_ok = true;
-            int32_t xb = 0;
+            for (int32_t i = lane; i < nlast; i += 32) {
+                int32_t ref[RX];
 #pragma unroll
-            for (int ax = 0; ax < RX; ++ax) {
-                ref[ax] -= int32_t(mdiv(uint32_t(ref[ax]), cd.mX_mul[ax], cd.mX_sh[ax])) * cd.sX[ax];
-                in_ok &= ref[ax] + cd.fmax_in1[ax] < cd.sX[ax];
-                xb += ref[ax] * cd.stX[ax];
-            }
-            int32_t x[kCP];
-            if (cd.contig1 && in_ok && (xb & 3) == 0 && xb + kCP <= cd.x_elems) {
-#pragma unroll
-                for (int v = 0; v < kCP / 4; ++v) {
-                    x[4 * v] = x[4 * v + 1] = x[4 * v + 2] = x[4 * v + 3] = 0;
-                    if (4 * v >= cd.n_in1) continue;
-                    const int4 q = __ldg(reinterpret_cast<const int4*>(X + xb) + v);
-                    x[4 * v] = q.x;
-                    x[4 * v + 1] = q.y;
-                    x[4 * v + 2] = q.z;
-                    x[4 * v + 3] = q.w;
-                }
-            } else {
-#pragma unroll
-                for (int p = 0; p < kCP; ++p) {
-                    x[p] = 0;
-                    if (p >= cd.n_in1) continue;
-                    int32_t off;
-                    if (in_ok) {
-                        off = xb + cd.lin_in1[p];
-                    } else {
-                        off = 0;
-#pragma unroll
-                        for (int ax = 0; ax < RX; ++ax) {
-                            int32_t c = ref[ax] + cd.f_in1[p][ax];   // toroidal pattern element
-                            if (c >= cd.sX[ax]) c -= cd.sX[ax];
-                            off += c * cd.stX[ax];
-                        }
-                    }
-                    x[p] = __ldg(X + off);
-                }
-            }
-            {   // prefix sums: window k = pre[start + len] - pre[start]
-                int32_t acc = 0;
-                my[0] = 0;
-#pragma unroll
-                for (int p = 0; p < kCP; ++p) {
-                    if (p >= cd.n_in1) continue;
-                    acc += x[p];
-                    my[(p + 1) * 256] = acc;
-                }
-            }
-            int32_t dbase = 0;   // box offset of the repetition's dense point R K (window offsets added below)
-#pragma unroll
-            for (int a = 0; a < RY; ++a) dbase += (Rraw[a] * cd.K[a] - g.v0[a]) * g.bst[a];
-            for (int k = 0; k < cd.nwin1; ++k) {
-                bool inside = true;
-                int32_t off = dbase;
-#pragma unroll
-                for (int a = 0; a < RY; ++a) {
-                    const int32_t dpos = Rraw[a] * cd.K[a] + cd.kk[k][a] - g.v0[a];
-                    inside &= dpos >= 0 && dpos < g.E[a];
-                    off += cd.kk[k][a] * g.bst[a];
-                }
-                if (!inside) continue;
-                const int32_t s0 = cd.start1[k];
-                box[off] = task_c(my[(s0 + cd.len1) * 256] - my[s0 * 256], cd.div1, cd.dv1_mul, cd.dv1_sh);
+                for (int ax = 0; ax < RX; ++ax) ref[ax] = rref[ax];
+                Rraw[RY - 1] = g.R0[RY - 1] + i;
+                chain_digits<RX>(cd, RY - 1, Rraw[RY - 1], ref);
+                chain_f1_rep<RX, RY, NP1>(cd, g, X, box, my, ref, Rraw);
             }
         }
         __syncthreads();
-        // ---- (2) f2 over the block's repetitions, patterns from the box, outputs to Z
-        const int32_t count = g.count, zb = g.zb;
-        for (int32_t e = threadIdx.x; e < count; e += 256) {
-            uint32_t rem = uint32_t(e);
-            int32_t boff = 0, zoff = zb;
+        // ---- (2) f2 over the block's repetitions: a warp per row (inner dims but the innermost), lanes along the
+        // innermost; patterns from the box, outputs to Z
+        const int32_t nin = cd.n_inr, llast = nin == 1 ? g.len0 : cd.in_len[nin - 1];
+        const int32_t nrow2 = g.count / llast, bl = g.bstep[nin - 1], zl = cd.in_z[nin - 1];
+        for (int32_t row = warp; row < nrow2; row += 8) {
+            uint32_t rem = uint32_t(row);
+            int32_t boff = 0, zoff = g.zb;
 #pragma unroll
-            for (int d = kCIn - 1; d >= 1; --d) {
-                if (d >= cd.n_inr) continue;
+            for (int d = kCIn - 2; d >= 1; --d) {
+                if (d >= nin - 1) continue;
                 const uint32_t q = mdiv(rem, cd.in_mul[d], cd.in_sh[d]);
                 const int32_t i = int32_t(rem - q * uint32_t(cd.in_len[d]));
                 rem = q;
                 boff += g.bstep[d] * i;
                 zoff += cd.in_z[d] * i;
             }
-            boff += g.bstep[0] * int32_t(rem);
-            zoff += cd.in_z[0] * int32_t(rem);
-            {
+            if (nin > 1) {
+                boff += g.bstep[0] * int32_t(rem);
+                zoff += cd.in_z[0] * int32_t(rem);
+            }
+            for (int32_t i = lane; i < llast; i += 32) {
+                const int32_t bo = boff + bl * i, zo = zoff + zl * i;
                 int32_t acc = 0;
                 my[0] = 0;
 #pragma unroll
                 for (int p = 0; p < kCP; ++p) {
                     if (p >= cd.n_in2) continue;
-                    acc += box[boff + g.poff[p]];
+                    acc += box[bo + g.poff[p]];
                     my[(p + 1) * 256] = acc;
                 }
-            }
-            for (int k = 0; k < cd.nwin2; ++k) {
-                const int32_t s0 = cd.start2[k];
-                Z[zoff + cd.zF[k]] = task_c(my[(s0 + cd.len2) * 256] - my[s0 * 256], cd.div2, cd.dv2_mul, cd.dv2_sh);
+                for (int k = 0; k < cd.nwin2; ++k) {
+                    const int32_t s0 = cd.start2[k];
+                    Z[zo + cd.zF[k]] = task_c(my[(s0 + cd.len2) * 256] - my[s0 * 256], cd.div2, cd.dv2_mul, cd.dv2_sh);
+                }
             }
         }
         __syncthreads();   // the box and g are rewritten by the next block
@@ -301,13 +344,28 @@ __global__ void __launch_bounds__(256) chain_kernel(const __grid_constant__ Chai
 
 using ChainFn = void (*)(const ChainDev, const int32_t*, int32_t*);
 
-ChainFn chain_kernel_for(int rx, int ry) {
-    static const ChainFn tab[4][4] = {
-        {chain_kernel<1, 1>, chain_kernel<1, 2>, chain_kernel<1, 3>, chain_kernel<1, 4>},
-        {chain_kernel<2, 1>, chain_kernel<2, 2>, chain_kernel<2, 3>, chain_kernel<2, 4>},
-        {chain_kernel<3, 1>, chain_kernel<3, 2>, chain_kernel<3, 3>, chain_kernel<3, 4>},
-        {chain_kernel<4, 1>, chain_kernel<4, 2>, chain_kernel<4, 3>, chain_kernel<4, 4>}};
-    return tab[rx - 1][ry - 1];
+template <int RX>
+ChainFn chain_kernel_ry(int ry, int np) {
+    const int q = (np + 3) / 4 - 1;   // pattern padded to 4, 8, 12 or 16 elements
+#define AOL_CHAIN_NP(RY) \
+    (q == 0 ? chain_kernel<RX, RY, 4> : q == 1 ? chain_kernel<RX, RY, 8> : q == 2 ? chain_kernel<RX, RY, 12> \
+                                                                             : chain_kernel<RX, RY, 16>)
+    switch (ry) {
+        case 1: return AOL_CHAIN_NP(1);
+        case 2: return AOL_CHAIN_NP(2);
+        case 3: return AOL_CHAIN_NP(3);
+        default: return AOL_CHAIN_NP(4);
+    }
+#undef AOL_CHAIN_NP
+}
+
+ChainFn chain_kernel_for(int rx, int ry, int np) {
+    switch (rx) {
+        case 1: return chain_kernel_ry<1>(ry, np);
+        case 2: return chain_kernel_ry<2>(ry, np);
+        case 3: return chain_kernel_ry<3>(ry, np);
+        default: return chain_kernel_ry<4>(ry, np);
+    }
 }
 
 int64_t emod(int64_t a, int64_t m) {
@@ -511,6 +569,14 @@ bool plan_chain(const aol_filter_t* f1, const aol_filter_t* f2, ChainDev* cd, in
                 v += std::llabs(sstep[d]) * dig;
             }
             cd->kk[k][a] = int32_t(v);
+        }
+    }
+    for (int a = 0; a < kCR; ++a) {
+        cd->kkmin[a] = 1 << 30;
+        cd->kkmax[a] = -(1 << 30);
+        for (int64_t k = 0; k < nwin; ++k) {
+            cd->kkmin[a] = std::min(cd->kkmin[a], cd->kk[k][a]);
+            cd->kkmax[a] = std::max(cd->kkmax[a], cd->kk[k][a]);
         }
     }
     // ---- f2 input side: blocks of repetitions over a box of Y
@@ -725,7 +791,7 @@ aol_status_t aol_filter_chain_apply(const aol_filter_t* f1, const aol_filter_t* 
     DeviceInfo dev;
     st = device_info(&dev);
     if (st != AOL_OK) return st;
-    const ChainFn kern = chain_kernel_for(cd.rx, cd.ry);
+    const ChainFn kern = chain_kernel_for(cd.rx, cd.ry, cd.n_in1);
     st = kernel_smem(reinterpret_cast<const void*>(kern), smem);
     if (st != AOL_OK) return st;
     const int per_sm = std::max(1, kernel_occupancy(reinterpret_cast<const void*>(kern), 256, smem));
