@@ -85,6 +85,9 @@ struct ChainBlk {
     int32_t poff[kCP];                               // box offset of f2 pattern element p (relative)
     int32_t kkoff[kCW];                              // box offset of f1 window k relative to its repetition
     int32_t nrow1;                                   // f1: rows of repetitions (all Y dims but the last)
+    uint32_t nl_mul, nl_sh;                          // magic division by nR[last] (f1 row length)
+    int32_t llast;                                   // f2 row length (innermost inner repetition dim)
+    uint32_t ll_mul, ll_sh;
 };
 
 __device__ __forceinline__ uint32_t mdiv(uint32_t n, uint32_t mul, uint32_t sh) { return (__umulhi(n, mul) + n) >> sh; }
@@ -166,6 +169,10 @@ __device__ void chain_block(const ChainDev& cd, int32_t blk, ChainBlk& g, int RY
         g.kkoff[k] = o;
     }
     g.nrow1 = g.nrep1 / g.nR[RY - 1];
+    g.nl_mul = g.nR_mul[RY - 1];
+    g.nl_sh = g.nR_sh[RY - 1];
+    g.llast = cd.n_inr == 1 ? g.len0 : cd.in_len[cd.n_inr - 1];
+    magic_dev(uint32_t(g.llast), g.ll_mul, g.ll_sh);
 }
 
 // f1's repetition with dense coordinates Rraw (per Y dim) at X reference point ref: gather its pattern, window
@@ -272,27 +279,34 @@ __global__ void __launch_bounds__(256) chain_kernel(const __grid_constant__ Chai
     int32_t* pre = sm;                          // [kCP + 1][256] per-thread prefix sums
     int32_t* box = pre + (kCP + 1) * 256;
     int32_t* my = pre + threadIdx.x;
-    const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
     for (int32_t blk = blockIdx.x; blk < cd.nblocks; blk += gridDim.x) {
         if (threadIdx.x == 0) chain_block(cd, blk, g, RY);
         __syncthreads();
-        // ---- (1) fill the box with f1: a warp per row of covering repetitions (all Y dims but the last fixed),
-        // lanes along the last Y dim's repetition range (coalesced X patterns)
-        const int32_t nrow1 = g.nrow1, nlast = g.nR[RY - 1];
-        for (int32_t row = warp; row < nrow1; row += 8) {
-            int32_t rref[RX], Rraw[RY];
+        // ---- (1) fill the box with f1 over the covering repetitions, flattened as (row, i): a row fixes every Y
+        // dim but the last (its digits decomposed once per row change), i runs along the last Y dim's range
+        // (consecutive threads: consecutive X patterns)
+        const int32_t nlast = g.nR[RY - 1], n1 = g.nrep1;
+        {
+            int32_t rref[RX], Rraw[RY], cur_row = -1;
 #pragma unroll
-            for (int ax = 0; ax < RX; ++ax) rref[ax] = cd.o1[ax];
-            uint32_t mm = uint32_t(row);
+            for (int a = 0; a < RY; ++a) Rraw[a] = 0;
+            for (int32_t e = threadIdx.x; e < n1; e += 256) {
+                const uint32_t row = mdiv(uint32_t(e), g.nl_mul, g.nl_sh);
+                const int32_t i = e - int32_t(row) * nlast;
+                if (int32_t(row) != cur_row) {
+                    cur_row = int32_t(row);
 #pragma unroll
-            for (int a = RY - 2; a >= 0; --a) {
-                const uint32_t q = mdiv(mm, g.nR_mul[a], g.nR_sh[a]);
-                const int32_t i = int32_t(mm - q * uint32_t(g.nR[a]));
-                mm = q;
-                Rraw[a] = g.R0[a] + i;
-                chain_digits<RX>(cd, a, Rraw[a], rref);
-            }
-            for (int32_t i = lane; i < nlast; i += 32) {
+                    for (int ax = 0; ax < RX; ++ax) rref[ax] = cd.o1[ax];
+                    uint32_t mm = row;
+#pragma unroll
+                    for (int a = RY - 2; a >= 0; --a) {
+                        const uint32_t q = mdiv(mm, g.nR_mul[a], g.nR_sh[a]);
+                        const int32_t ia = int32_t(mm - q * uint32_t(g.nR[a]));
+                        mm = q;
+                        Rraw[a] = g.R0[a] + ia;
+                        chain_digits<RX>(cd, a, Rraw[a], rref);
+                    }
+                }
                 int32_t ref[RX];
 #pragma unroll
                 for (int ax = 0; ax < RX; ++ax) ref[ax] = rref[ax];
@@ -302,27 +316,34 @@ __global__ void __launch_bounds__(256) chain_kernel(const __grid_constant__ Chai
             }
         }
         __syncthreads();
-        // ---- (2) f2 over the block's repetitions: a warp per row (inner dims but the innermost), lanes along the
-        // innermost; patterns from the box, outputs to Z
-        const int32_t nin = cd.n_inr, llast = nin == 1 ? g.len0 : cd.in_len[nin - 1];
-        const int32_t nrow2 = g.count / llast, bl = g.bstep[nin - 1], zl = cd.in_z[nin - 1];
-        for (int32_t row = warp; row < nrow2; row += 8) {
-            uint32_t rem = uint32_t(row);
-            int32_t boff = 0, zoff = g.zb;
+        // ---- (2) f2 over the block's repetitions, flattened as (row, i) along the innermost inner dim; patterns
+        // from the box, outputs to Z
+        {
+            const int32_t nin = cd.n_inr, llast = g.llast, count = g.count;
+            const int32_t bl = g.bstep[nin - 1], zl = cd.in_z[nin - 1];
+            int32_t cur_row = -1, boff = 0, zoff = 0;
+            for (int32_t e = threadIdx.x; e < count; e += 256) {
+                const uint32_t row = mdiv(uint32_t(e), g.ll_mul, g.ll_sh);
+                const int32_t i = e - int32_t(row) * llast;
+                if (int32_t(row) != cur_row) {
+                    cur_row = int32_t(row);
+                    uint32_t rem = row;
+                    boff = 0;
+                    zoff = g.zb;
 #pragma unroll
-            for (int d = kCIn - 2; d >= 1; --d) {
-                if (d >= nin - 1) continue;
-                const uint32_t q = mdiv(rem, cd.in_mul[d], cd.in_sh[d]);
-                const int32_t i = int32_t(rem - q * uint32_t(cd.in_len[d]));
-                rem = q;
-                boff += g.bstep[d] * i;
-                zoff += cd.in_z[d] * i;
-            }
-            if (nin > 1) {
-                boff += g.bstep[0] * int32_t(rem);
-                zoff += cd.in_z[0] * int32_t(rem);
-            }
-            for (int32_t i = lane; i < llast; i += 32) {
+                    for (int d = kCIn - 2; d >= 1; --d) {
+                        if (d >= nin - 1) continue;
+                        const uint32_t q = mdiv(rem, cd.in_mul[d], cd.in_sh[d]);
+                        const int32_t id = int32_t(rem - q * uint32_t(cd.in_len[d]));
+                        rem = q;
+                        boff += g.bstep[d] * id;
+                        zoff += cd.in_z[d] * id;
+                    }
+                    if (nin > 1) {
+                        boff += g.bstep[0] * int32_t(rem);
+                        zoff += cd.in_z[0] * int32_t(rem);
+                    }
+                }
                 const int32_t bo = boff + bl * i, zo = zoff + zl * i;
                 int32_t acc = 0;
                 my[0] = 0;
