@@ -588,6 +588,7 @@ struct BoxDev {
     uint32_t in_mul[kBoxMaxInner], in_shift[kBoxMaxInner]; // magic division by in_len (dims >= 1)
     int32_t nblocks;
     int32_t pitch_pad;                                     // extra elements per smem box row
+    int32_t vec16;                                         // 1: rows load as 16-byte async copies (below)
 };
 
 __device__ __forceinline__ uint32_t magic_div(uint32_t n, uint32_t mul, uint32_t shift) {
@@ -603,6 +604,8 @@ struct BoxBlock {
     int32_t step[kBoxMaxInner];        // smem offset per unit of inner dim d
     int32_t off0;                      // smem offset of inner index 0
     int32_t rows, pitch;
+    int32_t phase;                     // vec16: box element x of a row sits at smem x + phase (same 16-byte phase as
+                                       // its global address)
 };
 
 __device__ __forceinline__ void box_block(const BoxDev& bd, int32_t blk, BoxBlock& b) {
@@ -648,7 +651,18 @@ __device__ __forceinline__ void box_block(const BoxDev& bd, int32_t blk, BoxBloc
         b.base[r] = v < 0 ? v + bd.ashape[r] : v;
         bstride[r] = st;
         if (r == 0) {
-            b.pitch = b.E[0] + bd.pitch_pad;
+            if (bd.vec16) {
+                // 16-byte async row copies: box element x sits at smem x + phase, the 16-byte phase of its global
+                // address (every row start has phase 0 and the row extent is a multiple of 16 bytes: host-checked);
+                // the pitch keeps row starts 16-byte aligned and is padded off multiples of 128 bytes
+                const int32_t V = bd.vec16;
+                b.phase = b.base[0] % V;
+                b.pitch = (b.E[0] + 2 * V - 2) / V * V;
+                if ((b.pitch * (16 / V)) % 128 == 0) b.pitch += V;
+            } else {
+                b.phase = 0;
+                b.pitch = b.E[0] + bd.pitch_pad;
+            }
             st = b.pitch;
         } else {
             st *= b.E[r];
@@ -656,6 +670,7 @@ __device__ __forceinline__ void box_block(const BoxDev& bd, int32_t blk, BoxBloc
         }
         b.off0 += -lo * bstride[r];   // smem offset of inner index 0
     }
+    b.off0 += b.phase;
 #pragma unroll
     for (int d = 0; d < kBoxMaxInner; ++d) {
         int32_t o = 0;
@@ -713,11 +728,33 @@ __device__ __forceinline__ void box_issue_load(const BoxDev& bd, const BoxBlock&
     for (int32_t row = warp; row < b.rows; row += 8) {
         const int32_t roff = box_row_offset(bd, b, row);
         if constexpr (ES >= 4) {
-            const uint32_t srow = ptx::smem_u32(buf) + uint32_t(row * b.pitch) * ES;
-            for (int32_t x = lane; x < El; x += 32) {
-                int32_t gc = c0 + x;
-                while (gc >= sl) gc -= sl;
-                ptx::cp_async<ES>(srow + uint32_t(x) * ES, A + roff + gc);
+            const uint32_t srow = ptx::smem_u32(buf) + uint32_t(row * b.pitch + b.phase) * ES;
+            if (bd.vec16) {
+                // the row as contiguous global segments (the wrap restarts at column 0), each copied as an unaligned
+                // head, 16-byte chunks and a tail; smem and global share the 16-byte phase
+                constexpr int32_t V = 16 / ES;
+                int32_t x = 0, gc = c0;
+                while (x < El) {
+                    const int32_t len = min(El - x, sl - gc);
+                    const int32_t head = min(len, (V - gc % V) % V);
+                    const int32_t nch = (len - head) / V;
+                    const int32_t tail = len - head - nch * V;
+                    const uint32_t sseg = srow + uint32_t(x) * ES;
+                    const T* gseg = A + roff + gc;
+                    if (lane < head) ptx::cp_async<ES>(sseg + uint32_t(lane) * ES, gseg + lane);
+                    for (int32_t c = lane; c < nch; c += 32)
+                        ptx::cp_async<16>(sseg + uint32_t(head + c * V) * ES, gseg + head + c * V);
+                    if (lane < tail)
+                        ptx::cp_async<ES>(sseg + uint32_t(head + nch * V + lane) * ES, gseg + head + nch * V + lane);
+                    x += len;
+                    gc = 0;
+                }
+            } else {
+                for (int32_t x = lane; x < El; x += 32) {
+                    int32_t gc = c0 + x;
+                    while (gc >= sl) gc -= sl;
+                    ptx::cp_async<ES>(srow + uint32_t(x) * ES, A + roff + gc);
+                }
             }
         } else {
             T* srow = reinterpret_cast<T*>(buf) + row * b.pitch;
@@ -855,7 +892,7 @@ __global__ void __launch_bounds__(256) tiler_box_kernel(const __grid_constant__ 
             T* A = static_cast<T*>(dst);
             for (int32_t row = warp; row < b.rows; row += 8) {
                 const int32_t roff = box_row_offset(bd, b, row);
-                const T* srow = box + row * b.pitch;
+                const T* srow = box + row * b.pitch + b.phase;
                 for (int32_t x = lane; x < El; x += 32) {
                     int32_t gc = c0 + x;
                     while (gc >= sl) gc -= sl;
@@ -977,8 +1014,17 @@ bool make_box(const TilerDev& td, int es, int mode, BoxDev* bd, int* smem_bytes,
     bd->tail_prod = int32_t(inner / lenk);
     magic32(bd->tail_prod, &bd->tail_mul, &bd->tail_shift);
     bd->pitch_pad = (E[ra - 1] % 32 == 0) ? 1 : 0;   // rows of 32-multiple length: odd pitch, fewer bank conflicts
+    // 16-byte async row copies: 4- or 8-byte elements, every row start 16-byte aligned (row strides and the
+    // row length multiples of 16 bytes) so that a box row shares its global addresses' 16-byte phase
+    if (es >= 4) {
+        const int V = 16 / es;
+        bool ok = td.ashape[ra - 1] % V == 0;
+        for (int a = 0; a < ra - 1; ++a) ok = ok && td.astride[a] % V == 0;
+        bd->vec16 = ok ? V : 0;
+    }
     const int64_t rows = vol / E[ra - 1];
-    const int64_t buf = (rows * (E[ra - 1] + bd->pitch_pad) * es + 15) / 16 * 16;
+    const int64_t pitch_max = bd->vec16 ? E[ra - 1] + 3 * bd->vec16 : E[ra - 1] + bd->pitch_pad;
+    const int64_t buf = (rows * pitch_max * es + 15) / 16 * 16;
     *buf_bytes = int(buf);
     *smem_bytes = int(((inner / lenk) * 4 + 15) / 16 * 16 + (mode == 0 ? 2 : 1) * buf);
     return true;
@@ -1280,6 +1326,8 @@ aol_status_t launch_v(const TilerDev& td, const void* src, void* dst, unsigned l
             // 16-byte vectors on the tile side when every block starts and ends on a 16-byte boundary
             constexpr int VW = 16 / ES;
             const void* tp = MODE == 0 ? dst : src;
+            const void* ap = MODE == 0 ? src : dst;   // the array side: 16-byte row copies need an aligned base
+            if (reinterpret_cast<uintptr_t>(ap) % 16) bd.vec16 = 0;
             bool vec = reinterpret_cast<uintptr_t>(tp) % 16 == 0 && (int64_t(bd.tail_prod) * ES) % 16 == 0;
             for (int d = 0; d < bd.n_out && vec; ++d) vec = (int64_t(bd.out_g[d]) * ES) % 16 == 0;
             auto kern = vec ? tiler_box_kernel<ES, VW, MODE> : tiler_box_kernel<ES, 1, MODE>;
