@@ -563,8 +563,8 @@ WrapTabDev make_wraptab(const Wrap32Dev& wd) {
 // tilers, ArrayOL single assignment).  Replaces the per-element offset arithmetic of the kernels above with
 // ~10 instructions per element and keeps both global sides streaming.
 constexpr int kBoxMaxInner = 4;           // inner dims (incl. the chunked one)
-constexpr int kBoxBytes = 36 * 1024;      // smem per box buffer (gather: two, + the offset table: 2 CTAs per SM)
-constexpr int kBoxTab = 8192;             // entries of the per-CTA inner offset table (32 KB)
+constexpr int kBoxBytes = 16 * 1024;      // smem per box buffer: small blocks, many CTAs per SM (a 36 KB box + 32 KB table ran 2 CTAs/SM, barrier-bound)
+constexpr int kBoxTab = 2048;             // entries of the per-CTA inner offset table (8 KB)
 
 // Array dims are stored REVERSED in the box descriptors (r = 0 is the innermost, contiguous array dim: the box
 // row), so that every per-dim array is indexed by compile-time constants after unrolling (registers, no local
