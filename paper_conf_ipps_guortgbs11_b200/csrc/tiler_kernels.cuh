@@ -563,8 +563,8 @@ WrapTabDev make_wraptab(const Wrap32Dev& wd) {
 // tilers, ArrayOL single assignment).  Replaces the per-element offset arithmetic of the kernels above with
 // ~10 instructions per element and keeps both global sides streaming.
 constexpr int kBoxMaxInner = 4;           // inner dims (incl. the chunked one)
-constexpr int kBoxBytes = 16 * 1024;      // smem per box buffer: small blocks, many CTAs per SM (a 36 KB box + 32 KB table ran 2 CTAs/SM, barrier-bound)
-constexpr int kBoxTab = 2048;             // entries of the per-CTA inner offset table (8 KB)
+constexpr int kBoxBytes = 36 * 1024;      // smem per box buffer (gather: two, + the offset table: 2 CTAs per SM; 16 KB boxes measured slower: barrier-bound)
+constexpr int kBoxTab = 8192;             // entries of the per-CTA inner offset table (32 KB)
 
 // Array dims are stored REVERSED in the box descriptors (r = 0 is the innermost, contiguous array dim: the box
 // row), so that every per-dim array is indexed by compile-time constants after unrolling (registers, no local
@@ -837,17 +837,28 @@ __global__ void __launch_bounds__(256) tiler_box_kernel(const __grid_constant__ 
             const T* box = reinterpret_cast<const T*>(bufs + (k & 1) * buf_bytes);
             T* Tg = static_cast<T*>(dst) + b.g0;
             const int32_t count = b.count, off0 = b.off0, step0 = b.step[0];
-            for (int32_t v = threadIdx.x; v * VW < count; v += 256) {
-                const uint32_t e = uint32_t(v * VW);
-                const uint32_t i0 = magic_div(e, bd.tail_mul, bd.tail_shift);
-                const int32_t t = int32_t(e - i0 * uint32_t(bd.tail_prod));
-                const int32_t o = off0 + step0 * int32_t(i0);
-                int32_t to[VW];
-                box_tab_vec<VW>(tab, t, to);
-                union { VT vec; T e[VW]; } pk;
+            // four independent vectors per thread per iteration: their table and data loads overlap (one vector
+            // at a time left the loop waiting on shared-memory latency)
+            constexpr int kU = 4;
+            for (int32_t v0 = threadIdx.x; v0 * VW < count; v0 += 256 * kU) {
+                int32_t o[kU], to[kU][VW];
 #pragma unroll
-                for (int j = 0; j < VW; ++j) pk.e[j] = box[o + to[j]];
-                reinterpret_cast<VT*>(Tg)[v] = pk.vec;
+                for (int u = 0; u < kU; ++u) {
+                    const int32_t v = min(v0 + 256 * u, count / VW - 1);
+                    const uint32_t e = uint32_t(v * VW);
+                    const uint32_t i0 = magic_div(e, bd.tail_mul, bd.tail_shift);
+                    const int32_t t = int32_t(e - i0 * uint32_t(bd.tail_prod));
+                    o[u] = off0 + step0 * int32_t(i0);
+                    box_tab_vec<VW>(tab, t, to[u]);
+                }
+                union { VT vec; T e[VW]; } pk[kU];
+#pragma unroll
+                for (int u = 0; u < kU; ++u)
+#pragma unroll
+                    for (int j = 0; j < VW; ++j) pk[u].e[j] = box[o[u] + to[u][j]];
+#pragma unroll
+                for (int u = 0; u < kU; ++u)
+                    if ((v0 + 256 * u) * VW < count) reinterpret_cast<VT*>(Tg)[v0 + 256 * u] = pk[u].vec;
             }
             __syncthreads();   // this buffer, its geometry slot and tab may be overwritten from here on
         }
@@ -874,19 +885,21 @@ __global__ void __launch_bounds__(256) tiler_box_kernel(const __grid_constant__ 
 #pragma unroll
                 for (int u = 0; u < kU; ++u)
                     if ((v0 + 256 * u) * VW < count) pk[u].vec = reinterpret_cast<const VT*>(Tg)[v0 + 256 * u];
+                int32_t o[kU], to[kU][VW];
 #pragma unroll
                 for (int u = 0; u < kU; ++u) {
-                    const int32_t v = v0 + 256 * u;
-                    if (v * VW >= count) continue;
+                    const int32_t v = min(v0 + 256 * u, count / VW - 1);
                     const uint32_t e = uint32_t(v * VW);
                     const uint32_t i0 = magic_div(e, bd.tail_mul, bd.tail_shift);
                     const int32_t t = int32_t(e - i0 * uint32_t(bd.tail_prod));
-                    const int32_t o = off0 + step0 * int32_t(i0);
-                    int32_t to[VW];
-                    box_tab_vec<VW>(tab, t, to);
-#pragma unroll
-                    for (int j = 0; j < VW; ++j) box[o + to[j]] = pk[u].e[j];
+                    o[u] = off0 + step0 * int32_t(i0);
+                    box_tab_vec<VW>(tab, t, to[u]);
                 }
+#pragma unroll
+                for (int u = 0; u < kU; ++u)
+                    if ((v0 + 256 * u) * VW < count)
+#pragma unroll
+                        for (int j = 0; j < VW; ++j) box[o[u] + to[u][j]] = pk[u].e[j];
             }
             __syncthreads();
             T* A = static_cast<T*>(dst);
