@@ -1,0 +1,31 @@
+#!/bin/bash
+# round 2 full run: every GPU test, smoke, the default bench (all records), variants, reference arm,
+# ncu launch list + full captures (headline i32, u8, u8->i16, every tiler / filter / chain kernel), sanitizers
+cd "$GRAFT_REPO_ROOT"
+mkdir -p gpurun_out
+T=${TAG:-r02_full}
+nvidia-smi --query-gpu=name,clocks.sm,clocks.max.sm,power.draw --format=csv > gpurun_out/${T}_gpu.txt 2>&1
+timeout 1500 python -m pytest tests -m gpu -q > gpurun_out/${T}_pytest_gpu.log 2>&1; echo "pytest rc=$?" >> gpurun_out/${T}_pytest_gpu.log
+timeout 300 python -c "import __graft_entry__ as g; g.smoke()" > gpurun_out/${T}_smoke.log 2>&1; echo "smoke rc=$?" >> gpurun_out/${T}_smoke.log
+timeout 900 python bench.py > gpurun_out/${T}_bench.json 2> gpurun_out/${T}_bench.err
+timeout 600 python bench.py --dtype u8 --no-cpu-baseline > gpurun_out/${T}_bench_u8.json 2>> gpurun_out/${T}_bench.err
+timeout 600 python bench.py --dtype u8 --out-dtype i16 --no-cpu-baseline > gpurun_out/${T}_bench_u8i16.json 2>> gpurun_out/${T}_bench.err
+timeout 600 python bench.py --dtype rgb8 --no-cpu-baseline > gpurun_out/${T}_bench_rgb8.json 2>> gpurun_out/${T}_bench.err
+timeout 600 python bench.py --impl reference --steps 3 --warmup 1 > gpurun_out/${T}_bench_reference.json 2>> gpurun_out/${T}_bench.err
+timeout 600 python tools/chain_probe.py > gpurun_out/${T}_chain.jsonl 2>> gpurun_out/${T}_bench.err
+timeout 600 ncu --metrics gpu__time_duration.sum --clock-control none --csv --log-file gpurun_out/${T}_launches.csv \
+    python bench.py --steps 3 --warmup 3 --no-e2e --no-cpu-baseline --extras none > gpurun_out/${T}_ncu_launch_bench.log 2>&1
+for v in "i32:" "u8:--dtype u8" "u8i16:--dtype u8 --out-dtype i16"; do
+  name=${v%%:*}; args=${v#*:}
+  timeout 900 ncu --set full --clock-control none --import-source on -k regex:fused_tma -s 3 -c 1 \
+      -o gpurun_out/${T}_${name} -f python bench.py --steps 1 --warmup 3 --no-e2e --no-cpu-baseline --extras none $args \
+      > gpurun_out/${T}_ncu_${name}.log 2>&1
+done
+timeout 900 ncu --set full --clock-control none --import-source on -k regex:"tiler|filter|chain" -c 40 \
+    -o gpurun_out/${T}_tiler -f python tools/tiler_probe_all.py > gpurun_out/${T}_ncu_tiler.log 2>&1
+timeout 900 ncu --set full --clock-control none --import-source on -k regex:"chain" -c 1 \
+    -o gpurun_out/${T}_chain -f python tools/chain_probe.py --ncu > gpurun_out/${T}_ncu_chain.log 2>&1
+for tool in memcheck synccheck; do
+  timeout 900 compute-sanitizer --tool $tool --error-exitcode 3 python tools/sanitize_workload.py > gpurun_out/${T}_sanitize_$tool.log 2>&1
+  echo "$tool rc=$?" >> gpurun_out/${T}_sanitize_summary.txt
+done

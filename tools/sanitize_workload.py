@@ -101,6 +101,26 @@ def main():
     y = aol.filter_apply(aol.filter_preset(aol.FILTER_H, P, H, W), x)
     z = aol.filter_apply(aol.filter_preset(aol.FILTER_V, P, H, 3 * W // 8), y)
     ok &= torch.equal(z, aol.downscale_frame(x.unsqueeze(1))[0][:, 0])
+    # round 2: the fused chain of the same two filters (one kernel), the box tiler kernels (wrapping blocking
+    # with 16-byte row copies and a ragged chunk; the paper's H input tiler), persistent plans
+    z2 = aol.filter_chain_apply(aol.filter_preset(aol.FILTER_H, P, H, W), aol.filter_preset(aol.FILTER_V, P, H, 3 * W // 8), x)
+    ok &= torch.equal(z, z2)
+    Ab = torch.arange(3 * 64 * 256, dtype=torch.int32, device="cuda").reshape(3, 64, 256)
+    tb = aol.make_tiler([3, 64, 256], [3, 8, 32], [8, 8], [1, 7, -9], [[1, 0, 0], [0, 8, 0], [0, 0, 8]], [[0, 0], [1, 0], [0, 1]])
+    Gb = aol.tiler_gather(tb, Ab)
+    Bb = torch.zeros_like(Ab)
+    aol.tiler_scatter(tb, Gb, Bb, mode="fast")
+    ok &= torch.equal(Ab, Bb)
+    Ac = torch.arange(50 * 1000, dtype=torch.int32, device="cuda").reshape(50, 1000)
+    tc = aol.make_tiler([50, 1000], [50, 125], [11], [3, -2], [[1, 0], [0, 8]], [[0], [1]])
+    aol.tiler_gather(tc, Ac)
+    xp = aol.synth_frames(4, 0, 2, 3, 36, 256)
+    pl = aol.FramePlan(xp, checksums=True)
+    zp, csp = pl.launch()
+    zq, csq = aol.downscale_frame(xp, checksums=True)
+    torch.cuda.synchronize()
+    ok &= torch.equal(zp, zq) and torch.equal(csp.view(torch.int64), csq.view(torch.int64))
+    pl.close()
     torch.cuda.synchronize()
     print("sanitize workload:", "OK" if ok else "MISMATCH")
     return 0 if ok else 1
