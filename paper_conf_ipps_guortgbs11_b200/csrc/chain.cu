@@ -175,11 +175,13 @@ __device__ void chain_block(const ChainDev& cd, int32_t blk, ChainBlk& g, int RY
     magic_dev(uint32_t(g.llast), g.ll_mul, g.ll_sh);
 }
 
-// f1's repetition with dense coordinates Rraw (per Y dim) at X reference point ref: gather its pattern, window
-// sums, task, and store the outputs that fall inside the box (all of them when `all_in`).
+// f1's repetition at X reference point ref: gather its pattern, window sums, task; store the outputs into the
+// box at dbase + kkoff[k] -- all of them when all_in, else only those whose dense position d0 + kk lies inside
+// the box on every Y dim.
 template <int RX, int RY, int NP1>
 __device__ __forceinline__ void chain_f1_rep(const ChainDev& cd, const ChainBlk& g, const int32_t* __restrict__ X,
-                                             int32_t* box, int32_t* my, int32_t (&ref)[RX], const int32_t (&Rraw)[RY]) {
+                                             int32_t* box, int32_t* my, int32_t (&ref)[RX], int32_t dbase,
+                                             bool all_in, const int32_t (&d0)[RY]) {
     bool in_ok = true;
     int32_t xb = 0;
 #pragma unroll
@@ -227,20 +229,12 @@ __device__ __forceinline__ void chain_f1_rep(const ChainDev& cd, const ChainBlk&
             my[(p + 1) * 256] = acc;
         }
     }
-    int32_t dbase = 0;
-    bool all_in = true;
-#pragma unroll
-    for (int a = 0; a < RY; ++a) {
-        const int32_t d0 = Rraw[a] * cd.K[a] - g.v0[a];
-        dbase += d0 * g.bst[a];
-        all_in &= d0 + cd.kkmin[a] >= 0 && d0 + cd.kkmax[a] < g.E[a];
-    }
     for (int k = 0; k < cd.nwin1; ++k) {
         if (!all_in) {
             bool inside = true;
 #pragma unroll
             for (int a = 0; a < RY; ++a) {
-                const int32_t dpos = Rraw[a] * cd.K[a] + cd.kk[k][a] - g.v0[a];
+                const int32_t dpos = d0[a] + cd.kk[k][a];
                 inside &= dpos >= 0 && dpos < g.E[a];
             }
             if (!inside) continue;
@@ -250,11 +244,13 @@ __device__ __forceinline__ void chain_f1_rep(const ChainDev& cd, const ChainBlk&
     }
 }
 
-// The f1 reference-point contribution of Y dim a's dense repetition coordinate Rraw (digits of R mod nRfull).
+// The f1 reference-point contribution of Y dim a's dense repetition coordinate Rraw (digits of R mod nRfull;
+// Rraw < 3 nRfull since the box spans less than two periods beyond its start).
 template <int RX>
 __device__ __forceinline__ void chain_digits(const ChainDev& cd, int a, int32_t Rraw, int32_t (&ref)[RX]) {
     uint32_t R = uint32_t(Rraw);
-    while (R >= uint32_t(cd.nRfull[a])) R -= uint32_t(cd.nRfull[a]);
+    if (R >= uint32_t(cd.nRfull[a])) R -= uint32_t(cd.nRfull[a]);
+    if (R >= uint32_t(cd.nRfull[a])) R -= uint32_t(cd.nRfull[a]);
 #pragma unroll
     for (int gg = 0; gg < kCDig; ++gg) {
         if (gg >= cd.nrd[a]) continue;
@@ -279,50 +275,67 @@ __global__ void __launch_bounds__(256) chain_kernel(const __grid_constant__ Chai
     int32_t* pre = sm;                          // [kCP + 1][256] per-thread prefix sums
     int32_t* box = pre + (kCP + 1) * 256;
     int32_t* my = pre + threadIdx.x;
+    const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
     for (int32_t blk = blockIdx.x; blk < cd.nblocks; blk += gridDim.x) {
         if (threadIdx.x == 0) chain_block(cd, blk, g, RY);
         __syncthreads();
         // ---- (1) fill the box with f1 over the covering repetitions, flattened as (row, i): a row fixes every Y
-        // dim but the last (its digits decomposed once per row change), i runs along the last Y dim's range
-        // (consecutive threads: consecutive X patterns)
+        // dim but the last, i runs along the last Y dim's range.  Each warp walks a contiguous range of the
+        // flattened index (lanes consecutive: coalesced X patterns), so a thread's row changes rarely and the row
+        // part (digits, reference point, box offset, inside test) is recomputed only then.
         const int32_t nlast = g.nR[RY - 1], n1 = g.nrep1;
         {
-            int32_t rref[RX], Rraw[RY], cur_row = -1;
+            const int32_t per_warp = (n1 + 8 * 32 - 1) / (8 * 32) * 32;
+            const int32_t e_end = min(n1, (warp + 1) * per_warp);
+            int32_t rref[RX], d0[RY], cur_row = -1, rbase = 0;
+            bool rin = true;
 #pragma unroll
-            for (int a = 0; a < RY; ++a) Rraw[a] = 0;
-            for (int32_t e = threadIdx.x; e < n1; e += 256) {
+            for (int a = 0; a < RY; ++a) d0[a] = 0;
+#pragma unroll
+            for (int ax = 0; ax < RX; ++ax) rref[ax] = 0;
+            for (int32_t e = warp * per_warp + lane; e < e_end; e += 32) {
                 const uint32_t row = mdiv(uint32_t(e), g.nl_mul, g.nl_sh);
                 const int32_t i = e - int32_t(row) * nlast;
                 if (int32_t(row) != cur_row) {
                     cur_row = int32_t(row);
 #pragma unroll
                     for (int ax = 0; ax < RX; ++ax) rref[ax] = cd.o1[ax];
+                    rbase = 0;
+                    rin = true;
                     uint32_t mm = row;
 #pragma unroll
                     for (int a = RY - 2; a >= 0; --a) {
                         const uint32_t q = mdiv(mm, g.nR_mul[a], g.nR_sh[a]);
                         const int32_t ia = int32_t(mm - q * uint32_t(g.nR[a]));
                         mm = q;
-                        Rraw[a] = g.R0[a] + ia;
-                        chain_digits<RX>(cd, a, Rraw[a], rref);
+                        const int32_t Rr = g.R0[a] + ia;
+                        chain_digits<RX>(cd, a, Rr, rref);
+                        d0[a] = Rr * cd.K[a] - g.v0[a];
+                        rbase += d0[a] * g.bst[a];
+                        rin &= d0[a] + cd.kkmin[a] >= 0 && d0[a] + cd.kkmax[a] < g.E[a];
                     }
                 }
                 int32_t ref[RX];
 #pragma unroll
                 for (int ax = 0; ax < RX; ++ax) ref[ax] = rref[ax];
-                Rraw[RY - 1] = g.R0[RY - 1] + i;
-                chain_digits<RX>(cd, RY - 1, Rraw[RY - 1], ref);
-                chain_f1_rep<RX, RY, NP1>(cd, g, X, box, my, ref, Rraw);
+                const int32_t Rl = g.R0[RY - 1] + i;
+                chain_digits<RX>(cd, RY - 1, Rl, ref);
+                d0[RY - 1] = Rl * cd.K[RY - 1] - g.v0[RY - 1];
+                const bool all_in = rin && d0[RY - 1] + cd.kkmin[RY - 1] >= 0 &&
+                                    d0[RY - 1] + cd.kkmax[RY - 1] < g.E[RY - 1];
+                chain_f1_rep<RX, RY, NP1>(cd, g, X, box, my, ref, rbase + d0[RY - 1] * g.bst[RY - 1], all_in, d0);
             }
         }
         __syncthreads();
-        // ---- (2) f2 over the block's repetitions, flattened as (row, i) along the innermost inner dim; patterns
-        // from the box, outputs to Z
+        // ---- (2) f2 over the block's repetitions, flattened as (row, i) along the innermost inner dim, warp-
+        // contiguous ranges as above; patterns from the box, outputs to Z
         {
             const int32_t nin = cd.n_inr, llast = g.llast, count = g.count;
             const int32_t bl = g.bstep[nin - 1], zl = cd.in_z[nin - 1];
+            const int32_t per_warp = (count + 8 * 32 - 1) / (8 * 32) * 32;
+            const int32_t e_end = min(count, (warp + 1) * per_warp);
             int32_t cur_row = -1, boff = 0, zoff = 0;
-            for (int32_t e = threadIdx.x; e < count; e += 256) {
+            for (int32_t e = warp * per_warp + lane; e < e_end; e += 32) {
                 const uint32_t row = mdiv(uint32_t(e), g.ll_mul, g.ll_sh);
                 const int32_t i = e - int32_t(row) * llast;
                 if (int32_t(row) != cur_row) {

@@ -15,16 +15,21 @@ timeout 600 python bench.py --impl reference --steps 3 --warmup 1 > gpurun_out/$
 timeout 600 python tools/chain_probe.py > gpurun_out/${T}_chain.jsonl 2>> gpurun_out/${T}_bench.err
 timeout 600 ncu --metrics gpu__time_duration.sum --clock-control none --csv --log-file gpurun_out/${T}_launches.csv \
     python bench.py --steps 3 --warmup 3 --no-e2e --no-cpu-baseline --extras none > gpurun_out/${T}_ncu_launch_bench.log 2>&1
+# ncu reports stay on the box (/tmp/ncu, tens of MB each); their raw metric pages come back as CSV
+mkdir -p /tmp/ncu
 for v in "i32:" "u8:--dtype u8" "u8i16:--dtype u8 --out-dtype i16"; do
   name=${v%%:*}; args=${v#*:}
   timeout 900 ncu --set full --clock-control none --import-source on -k regex:fused_tma -s 3 -c 1 \
-      -o gpurun_out/${T}_${name} -f python bench.py --steps 1 --warmup 3 --no-e2e --no-cpu-baseline --extras none $args \
+      -o /tmp/ncu/${T}_${name} -f python bench.py --steps 1 --warmup 3 --no-e2e --no-cpu-baseline --extras none $args \
       > gpurun_out/${T}_ncu_${name}.log 2>&1
+  ncu -i /tmp/ncu/${T}_${name}.ncu-rep --page raw --csv > gpurun_out/${T}_ncu_${name}_raw.csv 2>/dev/null
 done
-timeout 900 ncu --set full --clock-control none --import-source on -k regex:"tiler|filter|chain" -c 40 \
-    -o gpurun_out/${T}_tiler -f python tools/tiler_probe_all.py > gpurun_out/${T}_ncu_tiler.log 2>&1
-timeout 900 ncu --set full --clock-control none --import-source on -k regex:"chain" -c 1 \
-    -o gpurun_out/${T}_chain -f python tools/chain_probe.py --ncu > gpurun_out/${T}_ncu_chain.log 2>&1
+timeout 900 ncu --set full --clock-control none -k regex:"tiler|filter" -c 16 \
+    -o /tmp/ncu/${T}_tiler -f python tools/tiler_probe_all.py > gpurun_out/${T}_ncu_tiler.log 2>&1
+ncu -i /tmp/ncu/${T}_tiler.ncu-rep --page raw --csv > gpurun_out/${T}_ncu_tiler_raw.csv 2>/dev/null
+timeout 900 ncu --set full --clock-control none -k regex:"chain" -c 1 \
+    -o /tmp/ncu/${T}_chain -f python tools/chain_probe.py --ncu > gpurun_out/${T}_ncu_chain.log 2>&1
+ncu -i /tmp/ncu/${T}_chain.ncu-rep --page raw --csv > gpurun_out/${T}_ncu_chain_raw.csv 2>/dev/null
 for tool in memcheck synccheck; do
   timeout 900 compute-sanitizer --tool $tool --error-exitcode 3 python tools/sanitize_workload.py > gpurun_out/${T}_sanitize_$tool.log 2>&1
   echo "$tool rc=$?" >> gpurun_out/${T}_sanitize_summary.txt

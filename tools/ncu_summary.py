@@ -1,7 +1,7 @@
 #!/usr/bin/env python
 """Summarise an `ncu --set full` capture and a launch list into profiles/.
 
-usage: python tools/ncu_summary.py <prof.ncu-rep> <launches.csv|-> <tag> <workload-key> [<bench-log>]
+usage: python tools/ncu_summary.py <prof.ncu-rep|raw.csv> <launches.csv|-> <tag> <workload-key> [<bench-log>]
 Writes profiles/<tag>_ncu_full.txt, profiles/<tag>_launches.csv and merges the per-launch
 DRAM bytes into profiles/ncu_traffic.json (read by bench.py for roofline.traffic).  The entry is
 keyed by the source-tree hash and launch plan of the captured run, taken from the bench.py JSON
@@ -30,7 +30,12 @@ KEYS = [
 
 
 def raw(rep):
-    out = subprocess.run(["ncu", "-i", rep, "--page", "raw", "--csv"], capture_output=True, text=True).stdout
+    """The raw metric page: from a report (ncu -i) or from its CSV export (`ncu -i rep --page raw --csv`)."""
+    if rep.endswith(".csv"):
+        with open(rep) as f:
+            out = f.read()
+    else:
+        out = subprocess.run(["ncu", "-i", rep, "--page", "raw", "--csv"], capture_output=True, text=True).stdout
     rows = list(csv.reader(io.StringIO(out)))
     return rows[0], rows[1], rows[2:]
 
