@@ -134,7 +134,13 @@ def lib() -> ctypes.CDLL:
                               "(the CUDA library is required; there is no CPU fallback)")
         L = ctypes.CDLL(LIB_PATH)
         for name, (args, res) in SIGNATURES.items():
-            f = getattr(L, name)
+            f = getattr(L, name, None)
+            if f is None:
+                # only an older build loaded through AOL_LIB_PATH for an A/B can lack a symbol (the in-tree
+                # library exports every one: tests/test_abi.py); its callers then fail when they use it
+                if LIB_PATH != os.path.join(_HERE, "libaol.so"):
+                    continue
+                raise ImportError(f"{LIB_PATH} lacks {name}: rebuild it (make)")
             f.argtypes = args
             f.restype = res
         _lib = L

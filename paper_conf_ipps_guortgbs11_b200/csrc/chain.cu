@@ -245,12 +245,11 @@ __device__ __forceinline__ void chain_f1_rep(const ChainDev& cd, const ChainBlk&
 }
 
 // The f1 reference-point contribution of Y dim a's dense repetition coordinate Rraw (digits of R mod nRfull;
-// Rraw < 3 nRfull since the box spans less than two periods beyond its start).
+// a box taller than the Y dim -- small arrays, long patterns -- wraps Rraw around more than once).
 template <int RX>
 __device__ __forceinline__ void chain_digits(const ChainDev& cd, int a, int32_t Rraw, int32_t (&ref)[RX]) {
     uint32_t R = uint32_t(Rraw);
-    if (R >= uint32_t(cd.nRfull[a])) R -= uint32_t(cd.nRfull[a]);
-    if (R >= uint32_t(cd.nRfull[a])) R -= uint32_t(cd.nRfull[a]);
+    while (R >= uint32_t(cd.nRfull[a])) R -= uint32_t(cd.nRfull[a]);
 #pragma unroll
     for (int gg = 0; gg < kCDig; ++gg) {
         if (gg >= cd.nrd[a]) continue;

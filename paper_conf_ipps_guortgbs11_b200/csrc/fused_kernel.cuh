@@ -611,37 +611,36 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
             for (int off = 16; off > 0; off >>= 1) csacc += __shfl_xor_sync(0xffffffffu, csacc, off);
             if (lane == 0) red[tid >> 5] = csacc;
             ptx::named_bar_sync(2, NC);
-            if (tid < 32) {   // warp 0
-                unsigned long long sum = 0;
-                if (lane == 0)
+            const int64_t frame = plane / a.channels;
+            if (a.cs_mode == 0) {
+                if (tid == 0) {
+                    unsigned long long sum = 0;
                     for (int w = 0; w < NC / 32; ++w) sum += red[w];
-                const int64_t frame = plane / a.channels;
-                if (a.cs_mode == 0) {
                     // the checksums were zeroed by the preceding zero_checksums_kernel, which this launch may
                     // overlap (programmatic dependent launch): wait for it before the first atomic (no-op when
                     // the kernel was launched without the PDL attribute, and after the first wait)
-                    if (lane == 0) {
-                        ptx::griddep_wait();
-                        atomicAdd(reinterpret_cast<unsigned long long*>(a.cs + frame), sum);
-                    }
-                } else {
-                    unsigned last = 0;
-                    if (lane == 0) {
-                        a.cs_partial[u] = sum;
-                        __threadfence();   // the partial is visible before the count that publishes it
-                        last = atomicAdd(a.cs_count + frame, 1u) == unsigned(a.units_per_frame - 1) ? 1u : 0u;
-                    }
-                    if (__shfl_sync(0xffffffffu, last, 0)) {   // the frame's last unit: sum its partials
-                        __threadfence();
-                        const int64_t u0 = frame * a.units_per_frame;
-                        unsigned long long tot = 0;
-                        for (int32_t j = lane; j < a.units_per_frame; j += 32) tot += __ldcg(a.cs_partial + u0 + j);
+                    ptx::griddep_wait();
+                    atomicAdd(reinterpret_cast<unsigned long long*>(a.cs + frame), sum);
+                }
+            } else if (tid < 32) {   // plans: warp 0 publishes the unit's partial; the frame's last unit sums them
+                unsigned last = 0;
+                if (lane == 0) {
+                    unsigned long long sum = 0;
+                    for (int w = 0; w < NC / 32; ++w) sum += red[w];
+                    a.cs_partial[u] = sum;
+                    // release: the partial is visible to whoever observes the count; acquire: the last unit sees
+                    // every other unit's partial (one acq_rel atomic instead of two fences)
+                    last = ptx::atom_add_acq_rel_gpu(a.cs_count + frame, 1u) == unsigned(a.units_per_frame - 1) ? 1u : 0u;
+                }
+                if (__shfl_sync(0xffffffffu, last, 0)) {
+                    const int64_t u0 = frame * a.units_per_frame;
+                    unsigned long long tot = 0;
+                    for (int32_t j = lane; j < a.units_per_frame; j += 32) tot += __ldcg(a.cs_partial + u0 + j);
 #pragma unroll
-                        for (int off = 16; off > 0; off >>= 1) tot += __shfl_xor_sync(0xffffffffu, tot, off);
-                        if (lane == 0) {
-                            a.cs[frame] = tot;
-                            a.cs_count[frame] = 0u;   // ready for the next launch (stream-ordered after this grid)
-                        }
+                    for (int off = 16; off > 0; off >>= 1) tot += __shfl_xor_sync(0xffffffffu, tot, off);
+                    if (lane == 0) {
+                        a.cs[frame] = tot;
+                        a.cs_count[frame] = 0u;   // ready for the next launch (stream-ordered after this grid)
                     }
                 }
             }
