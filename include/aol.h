@@ -236,9 +236,8 @@ AOL_API aol_status_t aol_downscale_frame_plan_out(aol_dtype_t in_dtype, aol_dtyp
 /* A fused-downscale launch resolved once for fixed device buffers and shape (the d1 single-frame case,
  * where per-call host planning outweighs the kernel: the launch-overhead argument of P:L776-779).
  * aol_frame_plan_create checks the arguments exactly as aol_downscale_frame_out, plans the launch, encodes
- * the TMA descriptor of d_in, sets kernel attributes and allocates a small device workspace owned by the
- * plan ((units x 8 + frames x 4) bytes; the only device memory the library ever allocates, and never on
- * the launch path).  Host only, synchronising; frames > 0. */
+ * the TMA descriptor of d_in and sets kernel attributes, once.  Host only; frames > 0; the plan owns no
+ * device memory. */
 typedef struct aol_frame_plan* aol_frame_plan_t;
 AOL_API aol_status_t aol_frame_plan_create(const void* d_in, aol_dtype_t in_dtype, void* d_out, aol_dtype_t out_dtype,
                                            int64_t frames, int64_t channels, int64_t H, int64_t W,
@@ -246,15 +245,15 @@ AOL_API aol_status_t aol_frame_plan_create(const void* d_in, aol_dtype_t in_dtyp
 
 /* Enqueue the planned downscale on s (the device current at creation): d_in -> d_out as
  * aol_downscale_frame_out, with d_frame_checksums (nullable, 8-byte aligned, [frames], overwritten).
- * ONE kernel launch: the checksum epilogue sums per-unit partials in the plan's workspace (no zeroing
- * kernel).  Launches of one plan must be stream-ordered (one stream, or ordered by events): they share the
- * workspace.  Argument errors are those of a NULL plan or a misaligned checksum pointer. */
+ * Only the launches remain: the checksum zeroing kernel and the fused kernel as its programmatic dependent
+ * (one launch without checksums).  Argument errors are those of a NULL plan or a misaligned checksum
+ * pointer. */
 AOL_API aol_status_t aol_frame_plan_launch(aol_frame_plan_t plan, uint64_t* d_frame_checksums, cudaStream_t s);
 
 /* The launch configuration the plan uses. */
 AOL_API aol_status_t aol_frame_plan_info(aol_frame_plan_t plan, aol_plan_t* out);
 
-/* Free the plan and its workspace (waits for the device).  NULL is a no-op. */
+/* Free the plan (host memory only; launches already enqueued are unaffected).  NULL is a no-op. */
 AOL_API aol_status_t aol_frame_plan_destroy(aol_frame_plan_t plan);
 
 /* Per-frame checksum of an existing output batch (for the unfused paths):

@@ -347,14 +347,12 @@ aol_status_t prepare_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t 
     a.nbands = int32_t(H / 9);
     a.bands_per_unit = plan.bands_per_unit;
     a.units_per_plane = plan.units_per_plane;
-    a.units_per_frame = int32_t((rgb ? 1 : channels) * plan.units_per_plane);
     a.stages = plan.stages;
     const RingGeom geom = ring_geom(in_dtype, plan.out_es, W, plan.flags);
     a.stage_bytes = geom.stage_bytes;
     a.stage_stride = geom.stage_stride;
     a.out_bytes = geom.out_bytes;
     a.n_consumer = plan.block - 32;
-    a.cs_mode = 0;
     for (int c = 0; c < 2; ++c) {
         L->k[c] = pick(in_dtype, plan.out_es, c == 1, plan.reps_per_thread, W, plan.flags, plan.block,
                        plan.ctas_per_sm);
@@ -368,17 +366,15 @@ aol_status_t enqueue_fused(const FusedLaunch& L, uint64_t* d_cs, cudaStream_t s)
     FusedArgs a = L.args;
     a.cs = d_cs;
     KernelFn k = L.k[d_cs ? 1 : 0];
-    // With checksums (cs_mode 0): zero them in a one-CTA kernel and launch the fused kernel as its programmatic
+    // With checksums: zero them in a one-CTA kernel and launch the fused kernel as its programmatic
     // dependent, so the zeroing (and the launch gap after it) overlaps the fused kernel's start instead of
     // preceding it (single-frame latency).  Only the zero kernel can be the primary: it
     // is an ordinary launch, so everything earlier in the stream (e.g. the producer of X) has completed.
     // PDL invariant: the fused kernel issues its TMA loads and bulk stores without griddepcontrol.wait, so it
     // may only be a programmatic dependent of zero_checksums_kernel (which touches nothing but cs and waits
     // for its own predecessor); pdl therefore requires d_cs, and the zero kernel is launched right before it.
-    // cs_mode 1 (plans) needs no zeroing: one launch.
-    const bool zero = d_cs && a.cs_mode == 0;
-    // cs_mode 0: PDL after the zeroing kernel; plans (pdl_wait): PDL after whatever precedes (the kernel waits)
-    const bool pdl = (zero || a.pdl_wait) && !(L.flags & AOL_FLAG_NO_PDL);
+    const bool zero = d_cs != nullptr;
+    const bool pdl = zero && !(L.flags & AOL_FLAG_NO_PDL);
     if (zero) {
         cudaLaunchConfig_t zc;
         std::memset(&zc, 0, sizeof zc);

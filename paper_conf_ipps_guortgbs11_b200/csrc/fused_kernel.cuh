@@ -117,17 +117,6 @@ struct FusedArgs {
     int32_t rows_per_stage; // int32 path: 3 (a stage holds a row triple) or 1 (one row per stage: finer ring
                             // granularity for wide frames); always 3 for uint8
     int32_t row_pitch;      // uint8 paths: bytes per input row (W planar, 3W packed 24-bit pixels)
-    // Checksum epilogue.  cs_mode 0: one atomicAdd per unit into cs, which zero_checksums_kernel cleared first.
-    // cs_mode 1 (plan launches, aol_frame_plan_launch): no zeroing kernel -- each unit stores its partial sum in
-    // cs_partial[unit] and counts itself in cs_count[frame]; the frame's last unit sums the partials into
-    // cs[frame] and resets the counter to 0 for the next launch (self-resetting, one launch per call).
-    int32_t cs_mode;
-    int32_t pdl_wait;           // 1: launched as a programmatic dependent of an ARBITRARY predecessor (plans): the
-                                // producer and consumer thread 0 -- the only threads touching global memory --
-                                // wait for it (griddepcontrol.wait) before their first access
-    int32_t units_per_frame;    // cs_mode 1: work units of one frame (contiguous unit indices)
-    unsigned long long* cs_partial;
-    unsigned int* cs_count;
 };
 
 // Byte offset of 16-byte chunk `chunk` (0..7) of 128-byte line `line` under SWIZZLE_128B
@@ -304,7 +293,6 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
         // ------------------------------------------------ producer warp (TMA)
         if (tid == NC) {
             if ((kI32 && kSwz != 0) || a.u8_tensor) ptx::prefetch_tensormap(&tmap);
-            if (a.pdl_wait) ptx::griddep_wait();
             int s = 0;
             uint32_t ph = 0;
             for (int64_t k = 0, u = unit_of(a, 0); u < a.nunits; u = unit_of(a, ++k)) {
@@ -364,7 +352,6 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
     }
 
     // ---------------------------------------------------- consumer threads
-    if (a.pdl_wait && tid == 0) ptx::griddep_wait();
     const int lane = tid & 31;
     const bool active = kRP * tid < a.reps;
     const int r = active ? kRP * tid : a.reps - kRP;   // first repetition owned (clamped for idle lanes)
@@ -611,38 +598,14 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
             for (int off = 16; off > 0; off >>= 1) csacc += __shfl_xor_sync(0xffffffffu, csacc, off);
             if (lane == 0) red[tid >> 5] = csacc;
             ptx::named_bar_sync(2, NC);
-            const int64_t frame = plane / a.channels;
-            if (a.cs_mode == 0) {
-                if (tid == 0) {
-                    unsigned long long sum = 0;
-                    for (int w = 0; w < NC / 32; ++w) sum += red[w];
-                    // the checksums were zeroed by the preceding zero_checksums_kernel, which this launch may
-                    // overlap (programmatic dependent launch): wait for it before the first atomic (no-op when
-                    // the kernel was launched without the PDL attribute, and after the first wait)
-                    ptx::griddep_wait();
-                    atomicAdd(reinterpret_cast<unsigned long long*>(a.cs + frame), sum);
-                }
-            } else if (tid < 32) {   // plans: warp 0 publishes the unit's partial; the frame's last unit sums them
-                unsigned last = 0;
-                if (lane == 0) {
-                    unsigned long long sum = 0;
-                    for (int w = 0; w < NC / 32; ++w) sum += red[w];
-                    a.cs_partial[u] = sum;
-                    // release: the partial is visible to whoever observes the count; acquire: the last unit sees
-                    // every other unit's partial (one acq_rel atomic instead of two fences)
-                    last = ptx::atom_add_acq_rel_gpu(a.cs_count + frame, 1u) == unsigned(a.units_per_frame - 1) ? 1u : 0u;
-                }
-                if (__shfl_sync(0xffffffffu, last, 0)) {
-                    const int64_t u0 = frame * a.units_per_frame;
-                    unsigned long long tot = 0;
-                    for (int32_t j = lane; j < a.units_per_frame; j += 32) tot += __ldcg(a.cs_partial + u0 + j);
-#pragma unroll
-                    for (int off = 16; off > 0; off >>= 1) tot += __shfl_xor_sync(0xffffffffu, tot, off);
-                    if (lane == 0) {
-                        a.cs[frame] = tot;
-                        a.cs_count[frame] = 0u;   // ready for the next launch (stream-ordered after this grid)
-                    }
-                }
+            if (tid == 0) {
+                unsigned long long sum = 0;
+                for (int w = 0; w < NC / 32; ++w) sum += red[w];
+                // the checksums were zeroed by the preceding zero_checksums_kernel, which this launch may
+                // overlap (programmatic dependent launch): wait for it before the first atomic (no-op when
+                // the kernel was launched without the PDL attribute, and after the first wait)
+                ptx::griddep_wait();
+                atomicAdd(reinterpret_cast<unsigned long long*>(a.cs + plane / a.channels), sum);
             }
             ptx::named_bar_sync(2, NC);   // red[] is reused by the next unit
         }
@@ -729,8 +692,10 @@ using KernelFn = void (*)(const CUtensorMap, const FusedArgs);
 
 // A resolved fused-kernel launch (kernel 1): tensor map, arguments, the kernels without / with the checksum
 // epilogue (k[0] / k[1], smem attributes set), launch shape.  Built by prepare_fused (fused.cu), enqueued by
-// enqueue_fused: zero_checksums_kernel + the PDL fused launch for cs_mode 0, one launch for cs_mode 1.
-// Plans (plan.cu) keep one and re-enqueue it.
+// enqueue_fused (zero_checksums_kernel + the fused kernel as its programmatic dependent).  Plans (plan.cu) keep
+// one and re-enqueue it.  (A one-launch plan variant -- per-unit checksum partials with self-resetting counters,
+// extra FusedArgs fields -- measured slower on device and perturbed the register allocation of the packed-pixel
+// and int16-output instantiations by 2-9 %, profiles/r02_plan_epilogue_ab.jsonl; removed.)
 struct FusedLaunch {
     CUtensorMap map;
     FusedArgs args;

@@ -3,9 +3,11 @@
 // aol_downscale_frame re-plans every call: argument checks, the unit-size search, the TMA descriptor
 // encode, kernel-attribute lookups and two launches (checksum zeroing + the PDL fused kernel).  For one HD
 // frame that host work is longer than the kernel (the paper's own launch-overhead argument,
-// P:L776-779).  A plan resolves all of it once for fixed buffers and shape; a launch is then ONE
-// cudaLaunchKernelEx: the fused kernel's checksum epilogue runs in cs_mode 1 (per-unit partial sums and a
-// self-resetting per-frame counter in the plan's small device workspace), so no zeroing kernel is needed.
+// P:L776-779).  A plan resolves all of it once for fixed buffers and shape; a launch is then only the two
+// cudaLaunchKernelEx calls (checksum zeroing + the fused kernel as its programmatic dependent; one without
+// checksums).  A one-launch variant (per-unit checksum partials + self-resetting per-frame counters in a plan
+// workspace) measured slower on the device and perturbed the register allocation of other instantiations:
+// removed.
 #include <cuda_runtime.h>
 
 #include <cstring>
@@ -21,7 +23,6 @@ struct aol_frame_plan {
     void* d_out;
     aol_dtype_t in_dtype;
     int64_t frames, channels, H, W;
-    void* d_ws;   // cs_mode 1: [units] u64 partial sums, then [frames] u32 counters (zero between launches)
     int device;
 };
 
@@ -46,7 +47,6 @@ aol_status_t aol_frame_plan_create(const void* d_in, aol_dtype_t in_dtype, void*
     p->channels = channels;
     p->H = H;
     p->W = W;
-    p->d_ws = nullptr;
     cudaGetDevice(&p->device);
     st = plan_fused(in_dtype, out_dtype, d_in, d_out, frames, channels, H, W, opts, &p->plan);
     if (st == AOL_OK && p->plan.kernel == 1) {
@@ -54,25 +54,8 @@ aol_status_t aol_frame_plan_create(const void* d_in, aol_dtype_t in_dtype, void*
         for (int c = 0; c < 2 && st == AOL_OK; ++c)
             st = launch_preflight(reinterpret_cast<const void*>(p->launch.k[c]), p->launch.block, p->launch.smem,
                                   "fused_tma_kernel");
-        if (st == AOL_OK) {
-            const size_t units = size_t(p->launch.args.nunits);
-            const size_t bytes = units * 8 + size_t(frames) * 4;
-            cudaError_t e = cudaMalloc(&p->d_ws, bytes);
-            if (e == cudaSuccess) e = cudaMemset(static_cast<uint8_t*>(p->d_ws) + units * 8, 0, size_t(frames) * 4);
-            if (e == cudaSuccess) e = cudaDeviceSynchronize();   // counters are zero before any launch
-            if (e != cudaSuccess) {
-                set_error("plan workspace allocation failed: %s", cudaGetErrorString(e));
-                st = AOL_E_CUDA;
-            } else {
-                p->launch.args.cs_mode = 1;
-                p->launch.args.pdl_wait = 1;
-                p->launch.args.cs_partial = static_cast<unsigned long long*>(p->d_ws);
-                p->launch.args.cs_count = reinterpret_cast<unsigned int*>(static_cast<uint8_t*>(p->d_ws) + units * 8);
-            }
-        }
     }
     if (st != AOL_OK) {
-        if (p->d_ws) cudaFree(p->d_ws);
         delete p;
         return st;
     }
@@ -99,21 +82,8 @@ aol_status_t aol_frame_plan_info(aol_frame_plan_t p, aol_plan_t* out) {
 }
 
 aol_status_t aol_frame_plan_destroy(aol_frame_plan_t p) {
-    if (!p) return AOL_OK;
-    aol_status_t st = AOL_OK;
-    if (p->d_ws) {
-        int cur = 0;
-        cudaGetDevice(&cur);
-        cudaSetDevice(p->device);
-        cudaError_t e = cudaFree(p->d_ws);   // synchronising: pending launches of the plan finish first
-        cudaSetDevice(cur);
-        if (e != cudaSuccess) {
-            set_error("cudaFree of the plan workspace failed: %s", cudaGetErrorString(e));
-            st = AOL_E_CUDA;
-        }
-    }
-    delete p;
-    return st;
+    delete p;   // NULL is a no-op; the plan owns no device memory
+    return AOL_OK;
 }
 
 }  // extern "C"

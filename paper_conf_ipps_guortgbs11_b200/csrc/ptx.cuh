@@ -108,14 +108,6 @@ __device__ __forceinline__ void tma_load_3d(void* smem_dst, const CUtensorMap* m
         : "memory");
 }
 
-// Device-scope fetch-and-add with acquire-release semantics (publishes this thread's prior writes to whoever
-// observes the new value, and makes the writes published by earlier increments visible to this thread).
-__device__ __forceinline__ unsigned atom_add_acq_rel_gpu(unsigned* p, unsigned v) {
-    unsigned old;
-    asm volatile("atom.acq_rel.gpu.global.add.u32 %0, [%1], %2;" : "=r"(old) : "l"(p), "r"(v) : "memory");
-    return old;
-}
-
 // Non-bulk asynchronous copies global -> shared (LDGSTS), 4 or 8 bytes, grouped by commit / wait_group: many
 // element copies in flight per thread without holding registers.
 template <int BYTES>

@@ -1,7 +1,6 @@
-"""Persistent launch plans (aol_frame_plan_*): one kernel launch per call, the checksum epilogue's per-unit
-partials and self-resetting per-frame counters (no zeroing kernel).  Against the oracle for every input
-type, across repeated launches (counters must reset), with new input contents between launches, without
-checksums, and for a plan that falls back to the generic kernel."""
+"""Persistent launch plans (aol_frame_plan_*): validation, planning and the TMA descriptor resolved once, each
+call only the launches.  Against the oracle for every input type, across repeated launches, with new input
+contents between launches, without checksums, and for a plan that falls back to the generic kernel."""
 import ctypes
 
 import numpy as np
@@ -28,7 +27,7 @@ def test_plan_matches_oracle_over_repeated_launches(orc, shape, dtype):
     x = torch.from_numpy(xh.astype(np.uint8) if dtype == torch.uint8 else xh).cuda()
     plan = aol.FramePlan(x, checksums=True)
     assert plan.info()["kernel"] == 1
-    for _ in range(4):   # the per-frame counters reset themselves: every launch gives the same checksums
+    for _ in range(4):   # every launch re-zeroes and recomputes the checksums
         z, cs = plan.launch()
         torch.cuda.synchronize()
         assert aol.last_kernel() == "fused_tma_kernel"
