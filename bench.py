@@ -493,8 +493,9 @@ def record_d1(aol, peak, check):
                     "host_enqueue_us_per_call_python": plan_host_us,
                     "host_enqueue_us_per_call_c": c_enq["plan_launch_us"] if c_enq else None,
                     "same_outputs_as_downscale_frame": plan_ok,
-                    "note": "aol_frame_plan_launch: validation, planning and the TMA descriptor done once at "
-                            "creation; each call is the zeroing kernel + the fused kernel (PDL)"},
+                    "note": "aol_frame_plan_launch: validation, planning, the TMA descriptor and the launches "
+                            "(zeroing kernel + PDL fused kernel, recorded as a CUDA graph) done once at creation; "
+                            "each call is one cudaGraphLaunch"},
            "host_enqueue_us_per_call_c": c_enq["downscale_frame_us"] if c_enq else None,
            "frac_cold": (b / peak / 1e3) / (cold * 1e3), "frac_graph": (b / peak / 1e3) / (graph_ms * 1e3 / 20),
            "timing": "CUDA events, median of 50 (warm: 200 us GPU sleep before each call; cold: 512 MB fill before "

@@ -236,8 +236,8 @@ AOL_API aol_status_t aol_downscale_frame_plan_out(aol_dtype_t in_dtype, aol_dtyp
 /* A fused-downscale launch resolved once for fixed device buffers and shape (the d1 single-frame case,
  * where per-call host planning outweighs the kernel: the launch-overhead argument of P:L776-779).
  * aol_frame_plan_create checks the arguments exactly as aol_downscale_frame_out, plans the launch, encodes
- * the TMA descriptor of d_in and sets kernel attributes, once.  Host only; frames > 0; the plan owns no
- * device memory. */
+ * the TMA descriptor of d_in, sets kernel attributes and records the launches as a CUDA graph (on a private
+ * stream), once.  Host only; frames > 0; the plan allocates no buffers of its own. */
 typedef struct aol_frame_plan* aol_frame_plan_t;
 AOL_API aol_status_t aol_frame_plan_create(const void* d_in, aol_dtype_t in_dtype, void* d_out, aol_dtype_t out_dtype,
                                            int64_t frames, int64_t channels, int64_t H, int64_t W,
@@ -245,15 +245,15 @@ AOL_API aol_status_t aol_frame_plan_create(const void* d_in, aol_dtype_t in_dtyp
 
 /* Enqueue the planned downscale on s (the device current at creation): d_in -> d_out as
  * aol_downscale_frame_out, with d_frame_checksums (nullable, 8-byte aligned, [frames], overwritten).
- * Only the launches remain: the checksum zeroing kernel and the fused kernel as its programmatic dependent
- * (one launch without checksums).  Argument errors are those of a NULL plan or a misaligned checksum
- * pointer. */
+ * ONE cudaGraphLaunch of the recorded launches (checksum zeroing + the fused kernel as its programmatic
+ * dependent); the first call with a new checksum pointer records that graph first; into a stream that is
+ * being captured the two launches are enqueued directly.  Not thread-safe for one plan.  Argument errors are those of a NULL plan or a misaligned checksum pointer. */
 AOL_API aol_status_t aol_frame_plan_launch(aol_frame_plan_t plan, uint64_t* d_frame_checksums, cudaStream_t s);
 
 /* The launch configuration the plan uses. */
 AOL_API aol_status_t aol_frame_plan_info(aol_frame_plan_t plan, aol_plan_t* out);
 
-/* Free the plan (host memory only; launches already enqueued are unaffected).  NULL is a no-op. */
+/* Free the plan and its recorded graphs (launches already enqueued are unaffected).  NULL is a no-op. */
 AOL_API aol_status_t aol_frame_plan_destroy(aol_frame_plan_t plan);
 
 /* Per-frame checksum of an existing output batch (for the unfused paths):

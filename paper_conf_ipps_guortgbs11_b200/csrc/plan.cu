@@ -3,11 +3,12 @@
 // aol_downscale_frame re-plans every call: argument checks, the unit-size search, the TMA descriptor
 // encode, kernel-attribute lookups and two launches (checksum zeroing + the PDL fused kernel).  For one HD
 // frame that host work is longer than the kernel (the paper's own launch-overhead argument,
-// P:L776-779).  A plan resolves all of it once for fixed buffers and shape; a launch is then only the two
-// cudaLaunchKernelEx calls (checksum zeroing + the fused kernel as its programmatic dependent; one without
-// checksums).  A one-launch variant (per-unit checksum partials + self-resetting per-frame counters in a plan
-// workspace) measured slower on the device and perturbed the register allocation of other instantiations:
-// removed.
+// P:L776-779).  A plan resolves all of it once for fixed buffers and shape, and records the launches (checksum
+// zeroing + the fused kernel as its programmatic dependent; the fused kernel alone without checksums) as a CUDA
+// graph: a call is then ONE cudaGraphLaunch.  The graph for a checksum pointer is re-recorded only when the
+// caller passes a different one.  A one-launch variant (per-unit checksum partials + self-resetting per-frame
+// counters in a plan workspace) measured slower on the device and perturbed the register allocation of other
+// instantiations: removed.
 #include <cuda_runtime.h>
 
 #include <cstring>
@@ -24,9 +25,44 @@ struct aol_frame_plan {
     aol_dtype_t in_dtype;
     int64_t frames, channels, H, W;
     int device;
+    cudaStream_t cap = nullptr;                  // private stream the launches are recorded on
+    cudaGraphExec_t exec[2] = {nullptr, nullptr};  // [0] without checksums, [1] with checksums into graph_cs
+    uint64_t* graph_cs = nullptr;
 };
 
 using namespace aol;
+
+namespace {
+
+void drop_graph(cudaGraphExec_t& e) {
+    if (e) cudaGraphExecDestroy(e);
+    e = nullptr;
+}
+
+// Record the plan's launches for checksum pointer cs (nullptr: none) as an executable graph.
+aol_status_t record(aol_frame_plan* p, uint64_t* cs, cudaGraphExec_t* out) {
+    cudaError_t e = cudaStreamBeginCapture(p->cap, cudaStreamCaptureModeThreadLocal);
+    if (e != cudaSuccess) {
+        set_error("plan: stream capture failed to start: %s", cudaGetErrorString(e));
+        return AOL_E_CUDA;
+    }
+    const aol_status_t st = enqueue_fused(p->launch, cs, p->cap);
+    cudaGraph_t g = nullptr;
+    e = cudaStreamEndCapture(p->cap, &g);
+    if (st != AOL_OK) {
+        if (g) cudaGraphDestroy(g);
+        return st;
+    }
+    if (e == cudaSuccess) e = cudaGraphInstantiate(out, g, 0);
+    if (g) cudaGraphDestroy(g);
+    if (e != cudaSuccess) {
+        set_error("plan: recording the launches failed: %s", cudaGetErrorString(e));
+        return AOL_E_CUDA;
+    }
+    return AOL_OK;
+}
+
+}  // namespace
 
 extern "C" {
 
@@ -54,8 +90,18 @@ aol_status_t aol_frame_plan_create(const void* d_in, aol_dtype_t in_dtype, void*
         for (int c = 0; c < 2 && st == AOL_OK; ++c)
             st = launch_preflight(reinterpret_cast<const void*>(p->launch.k[c]), p->launch.block, p->launch.smem,
                                   "fused_tma_kernel");
+        if (st == AOL_OK) {
+            const cudaError_t e = cudaStreamCreateWithFlags(&p->cap, cudaStreamNonBlocking);
+            if (e != cudaSuccess) {
+                set_error("plan: stream creation failed: %s", cudaGetErrorString(e));
+                st = AOL_E_CUDA;
+            }
+        }
+        if (st == AOL_OK) st = record(p, nullptr, &p->exec[0]);
     }
     if (st != AOL_OK) {
+        drop_graph(p->exec[0]);
+        if (p->cap) cudaStreamDestroy(p->cap);
         delete p;
         return st;
     }
@@ -72,7 +118,29 @@ aol_status_t aol_frame_plan_launch(aol_frame_plan_t p, uint64_t* d_frame_checksu
                             d_frame_checksums, s);
     aol_status_t st = debug_injected_failure("fused_tma_kernel");
     if (st != AOL_OK) return st;
-    return enqueue_fused(p->launch, d_frame_checksums, s);
+    // a graph cannot be launched into a stream that is itself being captured (e.g. the caller records its own
+    // CUDA graph): enqueue the launches directly then -- they become nodes of the caller's graph
+    cudaStreamCaptureStatus cap = cudaStreamCaptureStatusNone;
+    if (cudaStreamIsCapturing(s, &cap) != cudaSuccess) {
+        set_error("plan: cudaStreamIsCapturing failed");
+        return AOL_E_CUDA;
+    }
+    if (cap != cudaStreamCaptureStatusNone) return enqueue_fused(p->launch, d_frame_checksums, s);
+    const int c = d_frame_checksums ? 1 : 0;
+    if (c && (!p->exec[1] || p->graph_cs != d_frame_checksums)) {   // first use of this checksum buffer
+        drop_graph(p->exec[1]);
+        p->graph_cs = nullptr;
+        st = record(p, d_frame_checksums, &p->exec[1]);
+        if (st != AOL_OK) return st;
+        p->graph_cs = d_frame_checksums;
+    }
+    const cudaError_t e = cudaGraphLaunch(p->exec[c], s);
+    note_launch("fused_tma_kernel");
+    if (e != cudaSuccess) {
+        set_error("plan: graph launch failed: %s", cudaGetErrorString(e));
+        return AOL_E_CUDA;
+    }
+    return AOL_OK;
 }
 
 aol_status_t aol_frame_plan_info(aol_frame_plan_t p, aol_plan_t* out) {
@@ -82,7 +150,11 @@ aol_status_t aol_frame_plan_info(aol_frame_plan_t p, aol_plan_t* out) {
 }
 
 aol_status_t aol_frame_plan_destroy(aol_frame_plan_t p) {
-    delete p;   // NULL is a no-op; the plan owns no device memory
+    if (!p) return AOL_OK;
+    drop_graph(p->exec[0]);
+    drop_graph(p->exec[1]);
+    if (p->cap) cudaStreamDestroy(p->cap);
+    delete p;
     return AOL_OK;
 }
 
