@@ -700,7 +700,7 @@ __device__ __forceinline__ int32_t box_row_offset(const BoxDev& bd, const BoxBlo
 // offset of its inner-dim-0 index: tab[t] = sum_{d >= 1} step[d] idx_d(t).  Built per CTA whenever the box
 // layout changes (only between a full and the ragged last chunk), so an element's box offset is then
 // off0 + step[0] i0 + tab[t]: one magic division per 16-byte vector and two shared loads per element.
-__device__ __forceinline__ void box_build_table(const BoxDev& bd, const BoxBlock& b, int32_t* tab) {
+__device__ __forceinline__ void box_build_table(const BoxDev& bd, const BoxBlock& b, int16_t* tab) {
     for (int32_t t = threadIdx.x; t < bd.tail_prod; t += blockDim.x) {
         uint32_t rem = uint32_t(t);
         int32_t off = 0;
@@ -711,7 +711,7 @@ __device__ __forceinline__ void box_build_table(const BoxDev& bd, const BoxBlock
             off += b.step[d] * int32_t(rem - q * uint32_t(bd.in_len[d]));
             rem = q;
         }
-        tab[t] = off;
+        tab[t] = int16_t(off);   // |off| < box elements <= 32767
     }
 }
 
@@ -779,62 +779,81 @@ __device__ __forceinline__ void box_issue_load(const BoxDev& bd, const BoxBlock&
 // The VW table entries of a 16-byte output vector (t is a multiple of VW): one 16-byte (or two / four) shared
 // load(s) instead of VW scalar ones (those hit the same bank group from every quarter-warp).
 template <int VW>
-__device__ __forceinline__ void box_tab_vec(const int32_t* tab, int32_t t, int32_t (&o)[VW]) {
-    if constexpr (VW % 4 == 0) {
+__device__ __forceinline__ void box_tab_vec(const int16_t* tab, int32_t t, int32_t (&o)[VW]) {
+    // VW int16 entries at t (a multiple of VW): one shared load of 2 VW bytes (two 16-byte loads for VW = 16)
+    if constexpr (VW >= 8) {
 #pragma unroll
-        for (int q = 0; q < VW / 4; ++q) {
-            const int4 v = *reinterpret_cast<const int4*>(tab + t + 4 * q);
-            o[4 * q] = v.x;
-            o[4 * q + 1] = v.y;
-            o[4 * q + 2] = v.z;
-            o[4 * q + 3] = v.w;
+        for (int q = 0; q < VW / 8; ++q) {
+            const int4 v = *reinterpret_cast<const int4*>(tab + t + 8 * q);
+            const uint32_t w[4] = {uint32_t(v.x), uint32_t(v.y), uint32_t(v.z), uint32_t(v.w)};
+#pragma unroll
+            for (int i = 0; i < 4; ++i) {
+                o[8 * q + 2 * i] = int32_t(int16_t(w[i] & 0xffffu));
+                o[8 * q + 2 * i + 1] = int32_t(w[i]) >> 16;
+            }
         }
-    } else if constexpr (VW == 2) {
+    } else if constexpr (VW == 4) {
         const int2 v = *reinterpret_cast<const int2*>(tab + t);
-        o[0] = v.x;
-        o[1] = v.y;
+        o[0] = int32_t(int16_t(uint32_t(v.x) & 0xffffu));
+        o[1] = v.x >> 16;
+        o[2] = int32_t(int16_t(uint32_t(v.y) & 0xffffu));
+        o[3] = v.y >> 16;
+    } else if constexpr (VW == 2) {
+        const int32_t v = *reinterpret_cast<const int32_t*>(tab + t);
+        o[0] = int32_t(int16_t(uint32_t(v) & 0xffffu));
+        o[1] = v >> 16;
     } else {
         o[0] = tab[t];
     }
 }
 
-// smem: [tail_prod] int32 offset table, then one box buffer (FAST scatter) or two (gather: the next block's box
-// loads asynchronously while the current one is written out), each 16-byte aligned.  A block's geometry is
+// smem: [tail_prod] int16 offset table, then one box buffer (FAST scatter; gather with nbuf = 1) or two (gather,
+// nbuf = 2: the next block's box loads asynchronously while the current one is written out), 16-byte aligned.  A block's geometry is
 // computed once, by thread 0, into shared memory (every thread computing it cost ~20 instructions per element).
 template <int ES, int VW, int MODE>
 __global__ void __launch_bounds__(256) tiler_box_kernel(const __grid_constant__ BoxDev bd, const void* __restrict__ src,
-                                                        void* __restrict__ dst, int32_t buf_bytes) {
+                                                        void* __restrict__ dst, int32_t buf_bytes, int32_t nbuf) {
     using T = typename Elem<ES>::T;
     using VT = typename Vec<ES * VW>::T;
     extern __shared__ __align__(16) uint8_t box_raw[];
     __shared__ BoxBlock geo[2];
-    int32_t* tab = reinterpret_cast<int32_t*>(box_raw);
-    uint8_t* bufs = box_raw + ((size_t(bd.tail_prod) * 4 + 15) & ~size_t(15));
+    int16_t* tab = reinterpret_cast<int16_t*>(box_raw);
+    uint8_t* bufs = box_raw + ((size_t(bd.tail_prod) * 2 + 15) & ~size_t(15));
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
     const int sl = bd.ashape[0];
     int32_t tab_len0 = -1;   // len0 the table was built for
     if (MODE == 0) {
-        // software pipeline over this CTA's blocks: box k+1 loads while box k is emitted
+        // nbuf = 2: software pipeline over this CTA's blocks, box k+1 loads while box k is emitted; nbuf = 1: one
+        // buffer (less smem, more CTAs per SM: the overlap comes from the other CTAs)
         int32_t blk = blockIdx.x;
         if (threadIdx.x == 0 && blk < bd.nblocks) box_block(bd, blk, geo[0]);
         __syncthreads();
-        if (blk < bd.nblocks) box_issue_load<ES>(bd, geo[0], src, bufs);
+        if (nbuf == 2 && blk < bd.nblocks) box_issue_load<ES>(bd, geo[0], src, bufs);
         ptx::cp_async_commit();
         for (int32_t k = 0; blk < bd.nblocks; ++k, blk += gridDim.x) {
             const int32_t nxt = blk + gridDim.x;
-            BoxBlock& gn = geo[(k + 1) & 1];
-            const BoxBlock& b = geo[k & 1];
-            if (threadIdx.x == 0 && nxt < bd.nblocks) box_block(bd, nxt, gn);
-            __syncthreads();
-            if (nxt < bd.nblocks) box_issue_load<ES>(bd, gn, src, bufs + ((k + 1) & 1) * buf_bytes);
-            ptx::cp_async_commit();
+            const int slot = nbuf == 2 ? (k & 1) : 0;
+            const BoxBlock& b = geo[slot];
+            if (nbuf == 2) {
+                BoxBlock& gn = geo[(k + 1) & 1];
+                if (threadIdx.x == 0 && nxt < bd.nblocks) box_block(bd, nxt, gn);
+                __syncthreads();
+                if (nxt < bd.nblocks) box_issue_load<ES>(bd, gn, src, bufs + ((k + 1) & 1) * buf_bytes);
+                ptx::cp_async_commit();
+            } else {
+                box_issue_load<ES>(bd, b, src, bufs);
+                ptx::cp_async_commit();
+            }
             if (b.len0 != tab_len0) {   // uniform across the CTA; the previous block's reads of tab have finished
                 box_build_table(bd, b, tab);
                 tab_len0 = b.len0;
             }
-            ptx::cp_async_wait<1>();   // this block's box has landed (the next one may still be in flight)
+            if (nbuf == 2)
+                ptx::cp_async_wait<1>();   // this block's box has landed (the next one may still be in flight)
+            else
+                ptx::cp_async_wait<0>();
             __syncthreads();
-            const T* box = reinterpret_cast<const T*>(bufs + (k & 1) * buf_bytes);
+            const T* box = reinterpret_cast<const T*>(bufs + slot * buf_bytes);
             T* Tg = static_cast<T*>(dst) + b.g0;
             const int32_t count = b.count, off0 = b.off0, step0 = b.step[0];
             // four independent vectors per thread per iteration: their table and data loads overlap (one vector
@@ -861,6 +880,8 @@ __global__ void __launch_bounds__(256) tiler_box_kernel(const __grid_constant__ 
                     if ((v0 + 256 * u) * VW < count) reinterpret_cast<VT*>(Tg)[v0 + 256 * u] = pk[u].vec;
             }
             __syncthreads();   // this buffer, its geometry slot and tab may be overwritten from here on
+            if (nbuf == 1 && threadIdx.x == 0 && nxt < bd.nblocks) box_block(bd, nxt, geo[0]);
+            if (nbuf == 1) __syncthreads();
         }
         ptx::cp_async_wait<0>();
     } else {
@@ -945,7 +966,7 @@ bool make_box(const TilerDev& td, int es, int mode, BoxDev* bd, int* smem_bytes,
         }
         return vol;
     };
-    const int64_t budget = kBoxBytes / es;
+    const int64_t budget = std::min<int64_t>(kBoxBytes / es, 32767 - 4 * 32);   // int16 table offsets
     // grow the inner block from the innermost dim outwards while the box fits; the first dim that does not fit
     // entirely is chunked
     int k = nd - 1;
@@ -1039,7 +1060,7 @@ bool make_box(const TilerDev& td, int es, int mode, BoxDev* bd, int* smem_bytes,
     const int64_t pitch_max = bd->vec16 ? E[ra - 1] + 3 * bd->vec16 : E[ra - 1] + bd->pitch_pad;
     const int64_t buf = (rows * pitch_max * es + 15) / 16 * 16;
     *buf_bytes = int(buf);
-    *smem_bytes = int(((inner / lenk) * 4 + 15) / 16 * 16 + (mode == 0 ? 2 : 1) * buf);
+    *smem_bytes = int(((inner / lenk) * 2 + 15) / 16 * 16 + (mode == 0 ? 2 : 1) * buf);   // (2 buffers: see caller)
     return true;
 }
 
@@ -1344,11 +1365,23 @@ aol_status_t launch_v(const TilerDev& td, const void* src, void* dst, unsigned l
             bool vec = reinterpret_cast<uintptr_t>(tp) % 16 == 0 && (int64_t(bd.tail_prod) * ES) % 16 == 0;
             for (int d = 0; d < bd.n_out && vec; ++d) vec = (int64_t(bd.out_g[d]) * ES) % 16 == 0;
             auto kern = vec ? tiler_box_kernel<ES, VW, MODE> : tiler_box_kernel<ES, 1, MODE>;
-            st = kernel_smem(reinterpret_cast<const void*>(kern), box_smem);   // up to 72 KB (table + box)
+            // gathers: double-buffered boxes unless one buffer per CTA buys more CTAs per SM (AOL_TILER_BOX_NBUF
+            // forces 1 or 2 for A/B measurements)
+            int nbuf = MODE == 0 ? 2 : 1;
+            if (MODE == 0) {
+                const int one = box_smem - box_buf;
+                const int cps2 = kernel_occupancy(reinterpret_cast<const void*>(kern), 256, box_smem);
+                const int cps1 = kernel_occupancy(reinterpret_cast<const void*>(kern), 256, one);
+                if (cps2 < 3 && cps1 >= 2 * cps2) nbuf = 1;
+                const char* e = std::getenv("AOL_TILER_BOX_NBUF");
+                if (e && (e[0] == '1' || e[0] == '2')) nbuf = e[0] - '0';
+                if (nbuf == 1) box_smem = one;
+            }
+            st = kernel_smem(reinterpret_cast<const void*>(kern), box_smem);
             if (st != AOL_OK) return st;
             const int per_sm = std::max(1, kernel_occupancy(reinterpret_cast<const void*>(kern), 256, box_smem));
             const int gb = int(std::max<int64_t>(1, std::min<int64_t>(bd.nblocks, int64_t(dev.num_sms) * per_sm)));
-            kern<<<gb, 256, box_smem, s>>>(bd, src, dst, box_buf);
+            kern<<<gb, 256, box_smem, s>>>(bd, src, dst, box_buf, nbuf);
             AOL_LAUNCH_CHECK("tiler_box_kernel");
             return AOL_OK;
           }
