@@ -1365,14 +1365,15 @@ aol_status_t launch_v(const TilerDev& td, const void* src, void* dst, unsigned l
             bool vec = reinterpret_cast<uintptr_t>(tp) % 16 == 0 && (int64_t(bd.tail_prod) * ES) % 16 == 0;
             for (int d = 0; d < bd.n_out && vec; ++d) vec = (int64_t(bd.out_g[d]) * ES) % 16 == 0;
             auto kern = vec ? tiler_box_kernel<ES, VW, MODE> : tiler_box_kernel<ES, 1, MODE>;
-            // gathers: double-buffered boxes unless one buffer per CTA buys more CTAs per SM (AOL_TILER_BOX_NBUF
-            // forces 1 or 2 for A/B measurements)
+            // gathers: one box buffer per CTA whenever that buys more CTAs per SM (the overlap then comes from the
+            // other CTAs: H_IN 0.278 -> 0.220 ms, wrapping d3 0.145 -> 0.142, profiles/r02_box_nbuf_ab.jsonl), else
+            // double-buffered (AOL_TILER_BOX_NBUF forces 1 or 2 for A/B measurements)
             int nbuf = MODE == 0 ? 2 : 1;
             if (MODE == 0) {
                 const int one = box_smem - box_buf;
                 const int cps2 = kernel_occupancy(reinterpret_cast<const void*>(kern), 256, box_smem);
                 const int cps1 = kernel_occupancy(reinterpret_cast<const void*>(kern), 256, one);
-                if (cps2 < 3 && cps1 >= 2 * cps2) nbuf = 1;
+                if (cps1 > cps2) nbuf = 1;
                 const char* e = std::getenv("AOL_TILER_BOX_NBUF");
                 if (e && (e[0] == '1' || e[0] == '2')) nbuf = e[0] - '0';
                 if (nbuf == 1) box_smem = one;
