@@ -589,6 +589,8 @@ struct BoxDev {
     int32_t nblocks;
     int32_t pitch_pad;                                     // extra elements per smem box row
     int32_t vec16;                                         // 1: rows load as 16-byte async copies (below)
+    int32_t vs;                                            // 1: a 16-byte output vector's elements are 16 contiguous
+                                                           // smem bytes at one phase: 16-byte shared reads
 };
 
 __device__ __forceinline__ uint32_t magic_div(uint32_t n, uint32_t mul, uint32_t shift) {
@@ -658,7 +660,14 @@ __device__ __forceinline__ void box_block(const BoxDev& bd, int32_t blk, BoxBloc
                 const int32_t V = bd.vec16;
                 b.phase = b.base[0] % V;
                 b.pitch = (b.E[0] + 2 * V - 2) / V * V;
-                if ((b.pitch * (16 / V)) % 128 == 0) b.pitch += V;
+                if (bd.vs) {
+                    // 16-byte reads: rows 8 words (mod 32) apart, so a quarter-warp reading chunks of 4 consecutive
+                    // rows x 2 adjacent chunks hits 8 different bank groups (the d3 blocking's access shape)
+                    const int32_t wpe = 16 / V / 4 > 0 ? 16 / V / 4 : 1;   // 4-byte words per element (ES >= 4)
+                    while ((b.pitch * wpe) % 32 != 8) b.pitch += V;
+                } else if ((b.pitch * (16 / V)) % 128 == 0) {
+                    b.pitch += V;
+                }
             } else {
                 b.phase = 0;
                 b.pitch = b.E[0] + bd.pitch_pad;
@@ -871,10 +880,40 @@ __global__ void __launch_bounds__(256) tiler_box_kernel(const __grid_constant__ 
                     box_tab_vec<VW>(tab, t, to[u]);
                 }
                 union { VT vec; T e[VW]; } pk[kU];
+                if constexpr (ES >= 4 && VW * ES == 16) {
+                    if (bd.vs) {
+                        // the vector's elements are contiguous in smem at a block-uniform phase: one 16-byte read
+                        // (phase 0) or two and a selection
+                        const int32_t ph = b.phase;
 #pragma unroll
-                for (int u = 0; u < kU; ++u)
+                        for (int u = 0; u < kU; ++u) {
+                            const int32_t a0 = o[u] + to[u][0] - ph;   // 16-byte aligned
+                            const uint4 c0 = *reinterpret_cast<const uint4*>(box + a0);
+                            if (ph == 0) {
+                                pk[u].vec = *reinterpret_cast<const VT*>(&c0);
+                            } else {
+                                const uint4 c1 = *reinterpret_cast<const uint4*>(box + a0 + VW);
+                                const uint32_t w[8] = {c0.x, c0.y, c0.z, c0.w, c1.x, c1.y, c1.z, c1.w};
+                                const int sh = ph * (ES / 4);   // in 4-byte words
+                                uint32_t r[4];
 #pragma unroll
-                    for (int j = 0; j < VW; ++j) pk[u].e[j] = box[o[u] + to[u][j]];
+                                for (int q = 0; q < 4; ++q)
+                                    r[q] = sh == 1 ? w[q + 1] : sh == 2 ? w[q + 2] : w[q + 3];
+                                pk[u].vec = *reinterpret_cast<const VT*>(r);
+                            }
+                        }
+                    } else {
+#pragma unroll
+                        for (int u = 0; u < kU; ++u)
+#pragma unroll
+                            for (int j = 0; j < VW; ++j) pk[u].e[j] = box[o[u] + to[u][j]];
+                    }
+                } else {
+#pragma unroll
+                    for (int u = 0; u < kU; ++u)
+#pragma unroll
+                        for (int j = 0; j < VW; ++j) pk[u].e[j] = box[o[u] + to[u][j]];
+                }
 #pragma unroll
                 for (int u = 0; u < kU; ++u)
                     if ((v0 + 256 * u) * VW < count) reinterpret_cast<VT*>(Tg)[v0 + 256 * u] = pk[u].vec;
@@ -1055,9 +1094,20 @@ bool make_box(const TilerDev& td, int es, int mode, BoxDev* bd, int* smem_bytes,
         bool ok = td.ashape[ra - 1] % V == 0;
         for (int a = 0; a < ra - 1; ++a) ok = ok && td.astride[a] % V == 0;
         bd->vec16 = ok ? V : 0;
+        // 16-byte shared reads of an output vector: the innermost inner dim walks the row (+1 per element) and
+        // its length is a multiple of V, every other inner dim steps the row by multiples of V (its steps along
+        // other array dims are multiples of the pitch, itself a multiple of V)
+        const int j_last = nd - 1;
+        bool vs = ok && (mode == 0) && td.ext[j_last] % V == 0 && (nd - k) >= 1;
+        for (int a = 0; a < ra && vs; ++a) {
+            const int64_t c = sc[j_last][a];
+            vs = (a == ra - 1) ? c == 1 : c == 0;
+        }
+        for (int d = k; d < j_last && vs; ++d) vs = sc[d][ra - 1] % V == 0;
+        bd->vs = vs ? 1 : 0;
     }
     const int64_t rows = vol / E[ra - 1];
-    const int64_t pitch_max = bd->vec16 ? E[ra - 1] + 3 * bd->vec16 : E[ra - 1] + bd->pitch_pad;
+    const int64_t pitch_max = bd->vec16 ? E[ra - 1] + 3 * bd->vec16 + (bd->vs ? 32 : 0) : E[ra - 1] + bd->pitch_pad;
     const int64_t buf = (rows * pitch_max * es + 15) / 16 * 16;
     *buf_bytes = int(buf);
     *smem_bytes = int(((inner / lenk) * 2 + 15) / 16 * 16 + (mode == 0 ? 2 : 1) * buf);   // (2 buffers: see caller)
@@ -1361,7 +1411,7 @@ aol_status_t launch_v(const TilerDev& td, const void* src, void* dst, unsigned l
             constexpr int VW = 16 / ES;
             const void* tp = MODE == 0 ? dst : src;
             const void* ap = MODE == 0 ? src : dst;   // the array side: 16-byte row copies need an aligned base
-            if (reinterpret_cast<uintptr_t>(ap) % 16) bd.vec16 = 0;
+            if (reinterpret_cast<uintptr_t>(ap) % 16) bd.vec16 = bd.vs = 0;
             bool vec = reinterpret_cast<uintptr_t>(tp) % 16 == 0 && (int64_t(bd.tail_prod) * ES) % 16 == 0;
             for (int d = 0; d < bd.n_out && vec; ++d) vec = (int64_t(bd.out_g[d]) * ES) % 16 == 0;
             auto kern = vec ? tiler_box_kernel<ES, VW, MODE> : tiler_box_kernel<ES, 1, MODE>;
