@@ -26,6 +26,7 @@
 #include <cstdint>
 #include <cstdlib>
 #include <cstring>
+#include <vector>
 
 #include "common.h"
 #include "ptx.cuh"
@@ -1123,6 +1124,240 @@ bool tiler_box_enabled() {
     return v;
 }
 
+// ------------------------------------------------------------ affine pieces of wrapping tilers
+// A wrapping tiler is affine on each region of its index space where no coordinate crosses the array edge.  When
+// every wrapping array dim is driven by at most two combined dims (an outer one and an inner one, used by no other
+// wrapping dim) and wraps at most once, those regions are a few boxes of the index space: for the outer index
+// values whose whole inner range stays inside (or wraps), one box; for the few boundary values, a split of the
+// inner range.  Each box is a LINEAR tiler on a sub-range (its own array base, the wrap folded in as -s_a *
+// stride_a), so the pieces run through the affine kernel's permuted walk with 16-byte vectors -- the d3 blocking
+// shifted to wrap in both image dims is 1 big piece + 8 slivers.  Pieces are cut into chunks; a CTA takes chunks
+// grid-stride and stages the chunk's piece constants in shared memory.
+constexpr int kMaxPieces = 16;
+constexpr int kPieceChunk = 4096;   // vectors per chunk
+
+struct PiecesDev {
+    int32_t nd, npieces, nchunks;
+    int32_t p_lin[2 * AOL_MAX_RANK], p_gst[2 * AOL_MAX_RANK];    // permuted strides (the parent's)
+    int32_t len[kMaxPieces][2 * AOL_MAX_RANK];                   // permuted extents of each piece
+    uint32_t mul[kMaxPieces][2 * AOL_MAX_RANK], shift[kMaxPieces][2 * AOL_MAX_RANK];
+    int32_t abase[kMaxPieces], tbase[kMaxPieces];
+    int32_t nvec[kMaxPieces];                                    // vectors in the piece
+    int32_t chunk0[kMaxPieces + 1];                              // first chunk of each piece (prefix)
+};
+
+template <int ES, int V, int MODE>
+__global__ void __launch_bounds__(256) tiler_pieces_kernel(const __grid_constant__ PiecesDev pd,
+                                                           const void* __restrict__ src, void* __restrict__ dst) {
+    using T = typename Elem<ES>::T;
+    using VT = typename Vec<ES * V>::T;
+    __shared__ int4 pk[kND];      // {extent, magic multiplier, shift, array stride}
+    __shared__ int32_t pg[kND];   // tile stride
+    __shared__ int32_t cur_piece;
+    if (threadIdx.x == 0) cur_piece = -1;
+    for (int32_t c = blockIdx.x; c < pd.nchunks; c += gridDim.x) {
+        int pc = 0;
+        while (pc + 1 < pd.npieces && pd.chunk0[pc + 1] <= c) ++pc;
+        __syncthreads();   // the previous chunk's readers of pk / pg are done
+        if (pc != cur_piece) {
+            if (threadIdx.x < pd.nd) {
+                const int d = threadIdx.x;
+                pk[d] = make_int4(pd.len[pc][d], int32_t(pd.mul[pc][d]), int32_t(pd.shift[pc][d]), pd.p_lin[d]);
+                pg[d] = pd.p_gst[d];
+            }
+            __syncthreads();
+            if (threadIdx.x == 0) cur_piece = pc;
+        }
+        __syncthreads();
+        const int32_t v_begin = (c - pd.chunk0[pc]) * kPieceChunk;
+        const int32_t v_end = min(pd.nvec[pc], v_begin + kPieceChunk);
+        const int32_t ab = pd.abase[pc], tb = pd.tbase[pc];
+        constexpr int kU = 2;
+        for (int32_t v0 = v_begin + int32_t((threadIdx.x & ~31u) * kU + (threadIdx.x & 31u)); v0 < v_end;
+             v0 += 256 * kU) {
+            int32_t off[kU], g[kU];
+#pragma unroll
+            for (int u = 0; u < kU; ++u) {
+                const int32_t v = v0 + 32 * u;
+                uint32_t n = v < v_end ? uint32_t(v) * V : 0u;
+                int32_t o = ab, gg = tb;
+#pragma unroll 1
+                for (int d = pd.nd - 1; d >= 0; --d) {
+                    const int4 p = pk[d];
+                    const uint32_t q = (__umulhi(n, uint32_t(p.y)) + n) >> p.z;
+                    const int32_t i = int32_t(n - q * uint32_t(p.x));
+                    n = q;
+                    o += p.w * i;
+                    gg += pg[d] * i;
+                }
+                off[u] = o;
+                g[u] = gg;
+            }
+            VT val[kU];
+#pragma unroll
+            for (int u = 0; u < kU; ++u)
+                if (v0 + 32 * u < v_end)
+                    val[u] = reinterpret_cast<const VT*>(static_cast<const T*>(src) + (MODE == 0 ? off[u] : g[u]))[0];
+#pragma unroll
+            for (int u = 0; u < kU; ++u)
+                if (v0 + 32 * u < v_end)
+                    reinterpret_cast<VT*>(static_cast<T*>(dst) + (MODE == 0 ? g[u] : off[u]))[0] = val[u];
+        }
+    }
+}
+
+// One piece under construction: a sub-range per combined dim, a wrap flag per array dim.
+struct PieceBox {
+    int64_t start[2 * AOL_MAX_RANK], len[2 * AOL_MAX_RANK];
+    uint32_t wrapped;   // bit a: array dim a wrapped once inside this piece
+};
+
+// Split the parent tiler into affine pieces; false if it does not have the structure above (or needs more than
+// kMaxPieces pieces, or would not fit 31-bit offsets).  pieces_vec / pieces_scalar: pieces whose walk can use
+// V-element vectors, and the rest.
+bool make_pieces(const TilerDev& td, int es, const void* arr, const void* tiles, int V, PiecesDev* pv, PiecesDev* ps) {
+    if (td.linear || !td.fast32 || td.array_elems >= (int64_t(1) << 31) || td.total >= (int64_t(1) << 31)) return false;
+    const int nd = td.nd, ra = td.ra;
+    std::vector<PieceBox> boxes(1);
+    for (int d = 0; d < nd; ++d) {
+        boxes[0].start[d] = 0;
+        boxes[0].len[d] = td.ext[d];
+    }
+    boxes[0].wrapped = 0;
+    int used_by[2 * AOL_MAX_RANK];
+    for (int d = 0; d < nd; ++d) used_by[d] = -1;
+    for (int a = 0; a < ra; ++a) {
+        if ((td.nowrap_mask >> a) & 1) continue;
+        int ds[2], n = 0;
+        int64_t maxraw = td.org[a];
+        for (int d = 0; d < nd; ++d) {
+            if (td.coef[a][d] == 0 || td.ext[d] == 1) continue;
+            if (n == 2 || used_by[d] >= 0) return false;
+            used_by[d] = a;
+            ds[n++] = d;
+            maxraw += td.coef[a][d] * (td.ext[d] - 1);
+        }
+        if (n == 0 || maxraw >= 2 * td.ashape[a]) return false;   // at most one wrap
+        if (n == 2 && td.coef[a][ds[0]] < td.coef[a][ds[1]]) std::swap(ds[0], ds[1]);   // ds[0] outer
+        const int64_t T = td.ashape[a] - td.org[a];   // wrap iff sum of coef * idx >= T
+        std::vector<PieceBox> next;
+        for (const PieceBox& b : boxes) {
+            auto push = [&](int64_t s0, int64_t l0, int64_t s1, int64_t l1, bool w) {
+                if (l0 <= 0 || (n == 2 && l1 <= 0)) return;
+                PieceBox q = b;
+                q.start[ds[0]] = s0;
+                q.len[ds[0]] = l0;
+                if (n == 2) {
+                    q.start[ds[1]] = s1;
+                    q.len[ds[1]] = l1;
+                }
+                if (w) q.wrapped |= 1u << a;
+                next.push_back(q);
+            };
+            const int64_t Co = td.coef[a][ds[0]], So = b.start[ds[0]], Lo = b.len[ds[0]];
+            if (n == 1) {
+                const int64_t istar = std::min(std::max<int64_t>((T + Co - 1) / Co, So), So + Lo);   // first wrapping index
+                push(So, istar - So, 0, 0, false);
+                push(istar, So + Lo - istar, 0, 0, true);
+                continue;
+            }
+            const int64_t Cn = td.coef[a][ds[1]], Sn = b.start[ds[1]], Ln = b.len[ds[1]];
+            // threshold on the inner index for outer value io: inner >= t(io) wraps, t non-increasing in io
+            auto t_of = [&](int64_t io) {
+                const int64_t r = T - Co * io;
+                const int64_t t = r <= 0 ? 0 : (r + Cn - 1) / Cn;
+                return std::min(std::max(t, Sn), Sn + Ln);
+            };
+            int64_t io = So;
+            while (io < So + Lo) {
+                const int64_t t = t_of(io);
+                int64_t j = io + 1;   // extend while the same inner split applies
+                while (j < So + Lo && t_of(j) == t) ++j;
+                push(io, j - io, Sn, t - Sn, false);
+                push(io, j - io, t, Sn + Ln - t, true);
+                io = j;
+            }
+        }
+        boxes.swap(next);
+        if (boxes.size() > size_t(2 * kMaxPieces)) return false;
+    }
+    // build the two piece tables
+    std::memset(pv, 0, sizeof *pv);
+    std::memset(ps, 0, sizeof *ps);
+    int64_t lin[2 * AOL_MAX_RANK], gst[2 * AOL_MAX_RANK];
+    {
+        int64_t g = 1;
+        for (int d = nd - 1; d >= 0; --d) {
+            gst[d] = g;
+            g *= td.ext[d];
+        }
+        for (int d = 0; d < nd; ++d) {
+            lin[d] = 0;
+            for (int a = 0; a < ra; ++a) lin[d] += td.coef[a][d] * td.astride[a];
+        }
+    }
+    // walk order: array strides ascending (innermost = smallest), broadcast dims outermost -- as make_tiler_dev
+    int order[2 * AOL_MAX_RANK];
+    for (int d = 0; d < nd; ++d) order[d] = d;
+    auto key = [&](int d) { return lin[d] == 0 ? INT64_MAX : lin[d]; };
+    for (int i = 1; i < nd; ++i)
+        for (int j = i; j > 0 && key(order[j - 1]) < key(order[j]); --j) std::swap(order[j - 1], order[j]);
+    if (nd > 0 && lin[nd - 1] == 1) {
+        int pos = 0;
+        while (order[pos] != nd - 1) ++pos;
+        for (; pos < nd - 1; ++pos) order[pos] = order[pos + 1];
+        order[nd - 1] = nd - 1;
+    }
+    for (PiecesDev* P : {pv, ps}) {
+        P->nd = nd;
+        for (int i = 0; i < nd; ++i) {
+            P->p_lin[i] = int32_t(lin[order[i]]);
+            P->p_gst[i] = int32_t(gst[order[i]]);
+        }
+    }
+    const uintptr_t ptrs = reinterpret_cast<uintptr_t>(arr) | reinterpret_cast<uintptr_t>(tiles);
+    for (const PieceBox& b : boxes) {
+        int64_t count = 1, ab = 0, tb = 0;
+        for (int d = 0; d < nd; ++d) {
+            count *= b.len[d];
+            ab += lin[d] * b.start[d];
+            tb += gst[d] * b.start[d];
+        }
+        if (count == 0) continue;
+        for (int a = 0; a < ra; ++a) ab += (td.org[a] - (((b.wrapped >> a) & 1) ? td.ashape[a] : 0)) * td.astride[a];
+        // vectors: the innermost walked dim unit-stride on both sides, extents / bases / strides multiples of V
+        const int last = order[nd - 1];
+        bool vec = V > 1 && lin[last] == 1 && gst[last] == 1 && b.len[last] % V == 0 && ab % V == 0 && tb % V == 0 &&
+                   ptrs % uintptr_t(V * es) == 0;
+        for (int i = 0; i < nd - 1 && vec; ++i) vec = lin[order[i]] % V == 0 && gst[order[i]] % V == 0;
+        PiecesDev* P = vec ? pv : ps;
+        if (P->npieces == kMaxPieces) return false;
+        const int k = P->npieces++;
+        for (int i = 0; i < nd; ++i) {
+            P->len[k][i] = int32_t(b.len[order[i]]);
+            magic32(b.len[order[i]], &P->mul[k][i], &P->shift[k][i]);
+        }
+        P->abase[k] = int32_t(ab);
+        P->tbase[k] = int32_t(tb);
+        P->nvec[k] = int32_t(count / (vec ? V : 1));
+    }
+    for (PiecesDev* P : {pv, ps}) {
+        P->chunk0[0] = 0;
+        for (int k = 0; k < P->npieces; ++k) P->chunk0[k + 1] = P->chunk0[k] + (P->nvec[k] + kPieceChunk - 1) / kPieceChunk;
+        P->nchunks = P->chunk0[P->npieces];
+    }
+    return true;
+}
+
+// AOL_TILER_PIECES=0 disables the affine-piece path (A/B measurements only).
+bool tiler_pieces_enabled() {
+    static const bool v = [] {
+        const char* e = std::getenv("AOL_TILER_PIECES");
+        return !(e && e[0] == '0');
+    }();
+    return v;
+}
+
 // AOL_TILER_WRAPTAB=0 runs wrapping gathers / FAST scatters element by element (A/B measurements only).
 bool tiler_wraptab_enabled() {
     static const bool v = [] {
@@ -1400,6 +1635,33 @@ aol_status_t launch_v(const TilerDev& td, const void* src, void* dst, unsigned l
         return AOL_OK;
     }
     if constexpr (V == 1) {
+        if (MODE <= 1 && !lin && tiler_pieces_enabled()) {
+            constexpr int VV = 16 / ES;
+            PiecesDev pv, ps;
+            // only when (nearly) all elements run as 16-byte vectors: scalar pieces lose to the box kernel
+            bool use = make_pieces(td, ES, MODE == 0 ? src : dst, MODE == 0 ? dst : src, VV, &pv, &ps);
+            if (use) {
+                int64_t nv = 0;
+                for (int k = 0; k < pv.npieces; ++k) nv += int64_t(pv.nvec[k]) * VV;
+                use = 10 * nv >= 9 * td.total;
+            }
+            if (use) {
+                DeviceInfo dev;
+                aol_status_t st = device_info(&dev);
+                if (st != AOL_OK) return st;
+                if (pv.npieces > 0) {
+                    const int gp = int(std::max<int64_t>(1, std::min<int64_t>(pv.nchunks, int64_t(dev.num_sms) * 8)));
+                    if constexpr (VV > 1) tiler_pieces_kernel<ES, VV, MODE><<<gp, 256, 0, s>>>(pv, src, dst);
+                    AOL_LAUNCH_CHECK("tiler_pieces_kernel");
+                }
+                if (ps.npieces > 0) {
+                    const int gp = int(std::max<int64_t>(1, std::min<int64_t>(ps.nchunks, int64_t(dev.num_sms) * 8)));
+                    tiler_pieces_kernel<ES, 1, MODE><<<gp, 256, 0, s>>>(ps, src, dst);
+                    AOL_LAUNCH_CHECK("tiler_pieces_kernel");
+                }
+                return AOL_OK;
+            }
+        }
         BoxDev bd;
         int box_smem = 0, box_buf = 0;
         if (MODE <= 1 && !lin && tiler_box_enabled() && make_box(td, ES, MODE, &bd, &box_smem, &box_buf)) {

@@ -1,8 +1,9 @@
-"""The footprint-staged (box) tiler kernels against the oracle: wrapping gathers and FAST scatters whose
-array-side footprint per block of tiles is a dense box of whole rows -- the paper's H / V input tilers
-(Fig. 10, reading Z1), d3's wrapping blockings, negative coefficients, chunked
-blocks with a ragged last chunk, all element sizes.  Each case also checks which kernel ran
-(aol_debug_last_kernel), so the box path is known to be exercised."""
+"""The round-2 wrapping-tiler kernels against the oracle: the footprint-staged box kernel (gathers and FAST
+scatters whose array-side footprint per block of tiles is a dense box of whole rows) and the affine-piece kernel
+(wrapping tilers split into a few affine sub-boxes of the index space, each walked with 16-byte vectors) -- the
+paper's H / V input tilers (Fig. 10, reading Z1), d3's wrapping blockings, negative
+coefficients, chunked blocks with a ragged last chunk, all element sizes.  Each case also checks which kernel ran
+(aol_debug_last_kernel), so both paths are known to be exercised."""
 import numpy as np
 import pytest
 import torch
@@ -22,7 +23,10 @@ def _arr(rng, shape, es):
     return rng.integers(info.min // 2, info.max // 2, size=shape, dtype=np.int64).astype(NP[es])
 
 
-def _run(orc, arr, rep, pat, origin, P, F, es=4, seed=0, scatter=None, expect_box=True):
+STAGED = ("tiler_box_kernel", "tiler_pieces_kernel")
+
+
+def _run(orc, arr, rep, pat, origin, P, F, es=4, seed=0, scatter=None, expect_box=True, expect=STAGED):
     rng = np.random.default_rng(seed)
     A = _arr(rng, arr, es)
     t = aol.make_tiler(arr, rep, pat, origin, P, F)
@@ -33,7 +37,7 @@ def _run(orc, arr, rep, pat, origin, P, F, es=4, seed=0, scatter=None, expect_bo
     want = orc.gather(to, A)
     assert np.array_equal(G.cpu().numpy(), want)
     if expect_box:
-        assert kern == "tiler_box_kernel", kern
+        assert kern in expect, kern
     if scatter:
         Gs = _arr(rng, tuple(rep) + tuple(pat), es)
         B0 = _arr(rng, arr, es)
@@ -41,7 +45,7 @@ def _run(orc, arr, rep, pat, origin, P, F, es=4, seed=0, scatter=None, expect_bo
         aol.tiler_scatter(t, torch.from_numpy(Gs).cuda(), B, mode="fast")
         torch.cuda.synchronize()
         if expect_box:
-            assert aol.last_kernel() == "tiler_box_kernel", aol.last_kernel()
+            assert aol.last_kernel() in expect, aol.last_kernel()
         assert np.array_equal(B.cpu().numpy(), orc.scatter(to, Gs, B0))
     return kern
 
@@ -100,15 +104,37 @@ def test_random_wrapping_descriptors(orc, seed):
 
 
 def test_box_path_taken_by_the_paper_tilers():
-    """The d3 record's wrapping blocking and H_IN run the box kernel (the A/B in bench.py's d3 record)."""
+    """The d3 record's wrapping blocking runs as affine pieces (16-byte vectors), H_IN (11-element runs: no
+    vectors) through the box kernel."""
     A = torch.zeros((2, 64, 256), dtype=torch.int32, device="cuda")
     t = aol.make_tiler([2, 64, 256], [2, 8, 32], [8, 8], [0, -3, 5], [[1, 0, 0], [0, 8, 0], [0, 0, 8]],
                        [[0, 0], [1, 0], [0, 1]])
     aol.tiler_gather(t, A)
-    assert aol.last_kernel() == "tiler_box_kernel"
+    assert aol.last_kernel() == "tiler_pieces_kernel"
     X = torch.zeros((2, 36, 1920), dtype=torch.int32, device="cuda")
     th = aol.make_tiler([2, 36, 1920], [2, 36, 240], [11], [0, 0, 0], [[1, 0, 0], [0, 1, 0], [0, 0, 8]],
                         [[0], [0], [1]])
     aol.tiler_gather(th, X)
     assert aol.last_kernel() == "tiler_box_kernel"
     torch.cuda.synchronize()
+
+
+@pytest.mark.parametrize("es", [1, 2, 4, 8])
+@pytest.mark.parametrize("origin", [[0, -3, 5], [2, 13, -7], [0, 0, 1], [1, -8, 0]])
+def test_affine_pieces(orc, es, origin):
+    """Blockings shifted to wrap in one or both image dims split into affine pieces: gather and FAST scatter
+    against the oracle, the piece kernel asserted (vectors for the bulk, scalars for the slivers)."""
+    _run(orc, [3, 64, 256], [3, 8, 32], [8, 8], origin, [[1, 0, 0], [0, 8, 0], [0, 0, 8]],
+         [[0, 0], [1, 0], [0, 1]], es=es, scatter=True, expect=("tiler_pieces_kernel",))
+
+
+@pytest.mark.parametrize("seed", range(24))
+def test_affine_pieces_random_blockings(orc, seed):
+    """Random blockings (pattern = paving, or overlapping) with random origins and sizes, 4-byte elements."""
+    rng = np.random.default_rng(9500 + seed)
+    br, bc = int(rng.choice([1, 2, 4, 8])), int(rng.choice([4, 8, 16]))
+    nr, nc = int(rng.integers(1, 9)), int(rng.integers(2, 24))
+    arr = [2, br * nr, bc * nc]
+    org = [0, int(rng.integers(-br * nr, br * nr)), int(rng.integers(-bc * nc, bc * nc))]
+    _run(orc, arr, [2, nr, nc], [br, bc], org, [[1, 0, 0], [0, br, 0], [0, 0, bc]], [[0, 0], [1, 0], [0, 1]],
+         seed=seed, scatter=True, expect_box=False)
