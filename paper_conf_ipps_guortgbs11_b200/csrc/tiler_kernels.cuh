@@ -209,24 +209,29 @@ __global__ void __launch_bounds__(256) tiler_kernel(const TilerDev td, const voi
 }
 
 // Linear tilers whose array and tile offsets fit in 31 bits (the common case): the permuted walk with
-// all-32-bit digit arithmetic and the per-dimension constants staged once per CTA in shared memory
-// (one LDS.128 + one LDS per digit instead of five dynamically indexed constant-bank loads).
-template <int ES, int V, int MODE>
+// all-32-bit digit arithmetic, the per-dimension constants loaded once per thread into registers and the digit
+// loop fully unrolled for NDU dims (the tiler's, padded with unit extents on the outside): the walk's instruction
+// count is what bounds these kernels (round 2: a loop over constants staged in shared memory issued ~1.9x the
+// instructions; d3 affine gather 0.0878 ms there).
+template <int ES, int V, int MODE, int NDU>
 __global__ void __launch_bounds__(256) tiler_linear32_kernel(const TilerDev td, const void* __restrict__ src,
                                                              void* __restrict__ dst) {
     using T = typename Elem<ES>::T;
     using VT = typename Vec<ES * V>::T;
-    __shared__ int4 pk[kND];      // {extent, magic multiplier, shift, array stride}
-    __shared__ int32_t pg[kND];   // tile stride
-    if (threadIdx.x < td.nd) {
-        const int d = threadIdx.x;
-        pk[d] = make_int4(int32_t(td.p_ext[d]), int32_t(td.p_fd_mul[d]), int32_t(td.p_fd_shift[d]),
-                          int32_t(td.p_lin[d]));
-        pg[d] = int32_t(td.p_gst[d]);
+    int32_t L[NDU], AL[NDU], GS[NDU];
+    uint32_t M[NDU], S[NDU];
+#pragma unroll
+    for (int d = 0; d < NDU; ++d) {
+        const int e = d - (NDU - td.nd);
+        L[d] = e >= 0 ? int32_t(td.p_ext[e]) : 1;
+        M[d] = e >= 0 ? uint32_t(td.p_fd_mul[e]) : 0u;
+        S[d] = e >= 0 ? uint32_t(td.p_fd_shift[e]) : 0u;
+        AL[d] = e >= 0 ? int32_t(td.p_lin[e]) : 0;
+        GS[d] = e >= 0 ? int32_t(td.p_gst[e]) : 0;
     }
-    __syncthreads();
     const int32_t nvec = int32_t(td.total / V);
     const int32_t stride = int32_t(gridDim.x * blockDim.x);
+    const int32_t base = int32_t(td.base);
     // 2 vectors per thread per iteration with a 4x larger grid than the general kernels (tools/tiler_probe2.py,
     // profiles/r01_tiler_variants.jsonl: d3 gather 5.01 -> 5.22 TB/s; kU = 1, 4, 8 and grids x8..x512 are slower)
     constexpr int kU = 2;
@@ -237,16 +242,17 @@ __global__ void __launch_bounds__(256) tiler_linear32_kernel(const TilerDev td, 
         for (int u = 0; u < kU; ++u) {
             const int32_t v = v0 + 32 * u;
             uint32_t n = v < nvec ? uint32_t(v) * V : 0u;
-            int32_t o = int32_t(td.base), gg = 0;
-#pragma unroll 1
-            for (int d = td.nd - 1; d >= 0; --d) {
-                const int4 p = pk[d];
-                const uint32_t q = (__umulhi(n, uint32_t(p.y)) + n) >> p.z;
-                const int32_t i = int32_t(n - q * uint32_t(p.x));
+            int32_t o = base, gg = 0;
+#pragma unroll
+            for (int d = NDU - 1; d >= 1; --d) {
+                const uint32_t q = (__umulhi(n, M[d]) + n) >> S[d];
+                const int32_t i = int32_t(n - q * uint32_t(L[d]));
                 n = q;
-                o += p.w * i;
-                gg += pg[d] * i;
+                o += AL[d] * i;
+                gg += GS[d] * i;
             }
+            o += AL[0] * int32_t(n);   // the outermost digit is what is left (n < L[0] for every valid vector)
+            gg += GS[0] * int32_t(n);
             off[u] = o;
             g[u] = gg;
         }
@@ -1131,10 +1137,10 @@ bool tiler_box_enabled() {
 // values whose whole inner range stays inside (or wraps), one box; for the few boundary values, a split of the
 // inner range.  Each box is a LINEAR tiler on a sub-range (its own array base, the wrap folded in as -s_a *
 // stride_a), so the pieces run through the affine kernel's permuted walk with 16-byte vectors -- the d3 blocking
-// shifted to wrap in both image dims is 1 big piece + 8 slivers.  Pieces are cut into chunks; a CTA takes chunks
-// grid-stride and stages the chunk's piece constants in shared memory.
-constexpr int kMaxPieces = 16;
-constexpr int kPieceChunk = 4096;   // vectors per chunk
+// shifted to wrap in both image dims is 1 big piece + 8 slivers.  Pieces are cut into chunks of 1024 vectors, one
+// per CTA, which stages its piece's constants in shared memory (like the affine kernel's large grid).
+constexpr int kMaxPieces = 32;   // (a blocking wrapping in 3 dims: 3 x 3 x 2 = 18)
+constexpr int kPieceChunk = 1024;   // vectors per chunk (= per CTA: 2 iterations of 256 threads x 2 vectors)
 
 struct PiecesDev {
     int32_t nd, npieces, nchunks;
@@ -1143,67 +1149,178 @@ struct PiecesDev {
     uint32_t mul[kMaxPieces][2 * AOL_MAX_RANK], shift[kMaxPieces][2 * AOL_MAX_RANK];
     int32_t abase[kMaxPieces], tbase[kMaxPieces];
     int32_t nvec[kMaxPieces];                                    // vectors in the piece
+    int32_t phase[kMaxPieces];                                   // array-side misalignment (elements)
+    int32_t vec[kMaxPieces];                                     // 1: walked with vectors, 0: element by element
     int32_t chunk0[kMaxPieces + 1];                              // first chunk of each piece (prefix)
 };
 
-template <int ES, int V, int MODE>
-__global__ void __launch_bounds__(256) tiler_pieces_kernel(const __grid_constant__ PiecesDev pd,
-                                                           const void* __restrict__ src, void* __restrict__ dst) {
+// 16 bytes starting `b` bytes (0..15) into the 32 bytes (lo, hi): the misaligned array-side read of a vector
+// whose aligned neighbours were loaded instead (funnel shifts; b is uniform across the warp).
+__device__ __forceinline__ uint4 shift16(const uint4& lo, const uint4& hi, uint32_t b) {
+    const uint32_t w[8] = {lo.x, lo.y, lo.z, lo.w, hi.x, hi.y, hi.z, hi.w};
+    const uint32_t wb = b >> 2, sh = (b & 3u) * 8u;
+    uint32_t r[4];
+#pragma unroll
+    for (int q = 0; q < 4; ++q) {
+        const uint32_t a0 = wb == 0 ? w[q] : wb == 1 ? w[q + 1] : wb == 2 ? w[q + 2] : w[q + 3];
+        const uint32_t a1 = wb == 0 ? w[q + 1] : wb == 1 ? w[q + 2] : wb == 2 ? w[q + 3] : w[q + 4];
+        r[q] = __funnelshift_r(a0, a1, sh);
+    }
+    return make_uint4(r[0], r[1], r[2], r[3]);
+}
+
+// The walk of one chunk of a piece with W-element accesses (W = the vector width, or 1 for a piece that cannot
+// be vectorised), the digit constants in registers.
+template <int ES, int W, int MODE, int NDU>
+__device__ __forceinline__ void pieces_walk(const int32_t (&L)[NDU], const uint32_t (&M)[NDU], const uint32_t (&S)[NDU],
+                                            const int32_t (&AL)[NDU], const int32_t (&GS)[NDU], int32_t v_begin,
+                                            int32_t v_end, int32_t ab, int32_t tb, int32_t ph,
+                                            const void* __restrict__ src, void* __restrict__ dst) {
+    constexpr int V = W;
     using T = typename Elem<ES>::T;
     using VT = typename Vec<ES * V>::T;
-    __shared__ int4 pk[kND];      // {extent, magic multiplier, shift, array stride}
-    __shared__ int32_t pg[kND];   // tile stride
-    __shared__ int32_t cur_piece;
-    if (threadIdx.x == 0) cur_piece = -1;
-    for (int32_t c = blockIdx.x; c < pd.nchunks; c += gridDim.x) {
-        int pc = 0;
-        while (pc + 1 < pd.npieces && pd.chunk0[pc + 1] <= c) ++pc;
-        __syncthreads();   // the previous chunk's readers of pk / pg are done
-        if (pc != cur_piece) {
-            if (threadIdx.x < pd.nd) {
-                const int d = threadIdx.x;
-                pk[d] = make_int4(pd.len[pc][d], int32_t(pd.mul[pc][d]), int32_t(pd.shift[pc][d]), pd.p_lin[d]);
-                pg[d] = pd.p_gst[d];
-            }
-            __syncthreads();
-            if (threadIdx.x == 0) cur_piece = pc;
-        }
-        __syncthreads();
-        const int32_t v_begin = (c - pd.chunk0[pc]) * kPieceChunk;
-        const int32_t v_end = min(pd.nvec[pc], v_begin + kPieceChunk);
-        const int32_t ab = pd.abase[pc], tb = pd.tbase[pc];
-        constexpr int kU = 2;
-        for (int32_t v0 = v_begin + int32_t((threadIdx.x & ~31u) * kU + (threadIdx.x & 31u)); v0 < v_end;
-             v0 += 256 * kU) {
-            int32_t off[kU], g[kU];
+    const uint32_t lane = threadIdx.x & 31u;
+    constexpr int kU = 2;
+    for (int32_t v0 = v_begin + int32_t((threadIdx.x & ~31u) * kU + lane); v0 < v_end + int32_t(lane);
+         v0 += 256 * kU) {   // (whole warps iterate together: the realignment below shuffles)
+        int32_t off[kU], g[kU];
 #pragma unroll
-            for (int u = 0; u < kU; ++u) {
-                const int32_t v = v0 + 32 * u;
-                uint32_t n = v < v_end ? uint32_t(v) * V : 0u;
-                int32_t o = ab, gg = tb;
-#pragma unroll 1
-                for (int d = pd.nd - 1; d >= 0; --d) {
-                    const int4 p = pk[d];
-                    const uint32_t q = (__umulhi(n, uint32_t(p.y)) + n) >> p.z;
-                    const int32_t i = int32_t(n - q * uint32_t(p.x));
-                    n = q;
-                    o += p.w * i;
-                    gg += pg[d] * i;
-                }
-                off[u] = o;
-                g[u] = gg;
+        for (int u = 0; u < kU; ++u) {
+            const int32_t v = v0 + 32 * u;
+            uint32_t n = v < v_end ? uint32_t(v) * V : 0u;
+            int32_t o = ab, gg = tb;
+#pragma unroll
+            for (int d = NDU - 1; d >= 1; --d) {
+                const uint32_t q = (__umulhi(n, M[d]) + n) >> S[d];
+                const int32_t i = int32_t(n - q * uint32_t(L[d]));
+                n = q;
+                o += AL[d] * i;
+                gg += GS[d] * i;
             }
-            VT val[kU];
+            o += AL[0] * int32_t(n);   // the outermost digit is what is left (n < L[0] for every valid vector)
+            gg += GS[0] * int32_t(n);
+            off[u] = o;
+            g[u] = gg;
+        }
+        VT val[kU];
+        if constexpr (MODE == 0 && V * ES == 16) {
+            if (ph != 0) {
+                // array side misaligned by ph elements: each lane loads the aligned 16 bytes holding its vector's
+                // head; the tail comes from the next lane's load when that lane's vector follows on in the array
+                // (runs of tiles along a row), else from a second load of its own, issued together with the first
+                // (known from the decoded offsets alone).  Lanes past the end load the piece's first vector (in
+                // bounds) so that the whole warp takes part in the shuffles.
+                bool own[kU];
+#pragma unroll
+                for (int u = 0; u < kU; ++u) {
+                    const int32_t noff = __shfl_down_sync(0xffffffffu, off[u], 1);
+                    own[u] = v0 + 32 * u < v_end && (lane == 31 || noff != off[u] + V);
+                }
+                uint4 lo[kU], hi[kU];
+#pragma unroll
+                for (int u = 0; u < kU; ++u) {
+                    const uint4* a = reinterpret_cast<const uint4*>(static_cast<const T*>(src) + off[u] - ph);
+                    lo[u] = a[0];
+                    if (own[u]) hi[u] = a[1];
+                }
+#pragma unroll
+                for (int u = 0; u < kU; ++u) {
+                    uint4 h;
+                    h.x = __shfl_down_sync(0xffffffffu, lo[u].x, 1);
+                    h.y = __shfl_down_sync(0xffffffffu, lo[u].y, 1);
+                    h.z = __shfl_down_sync(0xffffffffu, lo[u].z, 1);
+                    h.w = __shfl_down_sync(0xffffffffu, lo[u].w, 1);
+                    if (!own[u]) hi[u] = h;
+                    const uint4 r = shift16(lo[u], hi[u], uint32_t(ph * ES));
+                    val[u] = *reinterpret_cast<const VT*>(&r);
+                }
+            } else {
+#pragma unroll
+                for (int u = 0; u < kU; ++u)
+                    if (v0 + 32 * u < v_end) val[u] = reinterpret_cast<const VT*>(static_cast<const T*>(src) + off[u])[0];
+            }
+        } else {
 #pragma unroll
             for (int u = 0; u < kU; ++u)
                 if (v0 + 32 * u < v_end)
                     val[u] = reinterpret_cast<const VT*>(static_cast<const T*>(src) + (MODE == 0 ? off[u] : g[u]))[0];
-#pragma unroll
-            for (int u = 0; u < kU; ++u)
-                if (v0 + 32 * u < v_end)
-                    reinterpret_cast<VT*>(static_cast<T*>(dst) + (MODE == 0 ? g[u] : off[u]))[0] = val[u];
         }
+        if constexpr (MODE == 1 && V * ES == 16) {
+            if (ph != 0) {
+                // array side misaligned by ph elements: lane L stores the aligned 16 bytes that start inside its
+                // vector (its last ph elements + the next lane's first V - ph) when the next lane's vector follows
+                // on in the array; a vector without such a neighbour stores its tail, one without an array-side
+                // predecessor its head, element by element.  Every element is stored exactly once.
+#pragma unroll
+                for (int u = 0; u < kU; ++u) {
+                    const bool valid = v0 + 32 * u < v_end;
+                    const uint4 lo = *reinterpret_cast<const uint4*>(&val[u]);
+                    uint4 hi;
+                    hi.x = __shfl_down_sync(0xffffffffu, lo.x, 1);
+                    hi.y = __shfl_down_sync(0xffffffffu, lo.y, 1);
+                    hi.z = __shfl_down_sync(0xffffffffu, lo.z, 1);
+                    hi.w = __shfl_down_sync(0xffffffffu, lo.w, 1);
+                    const int32_t noff = __shfl_down_sync(0xffffffffu, off[u], 1);
+                    const int32_t poff = __shfl_up_sync(0xffffffffu, off[u], 1);
+                    const bool nvalid = __shfl_down_sync(0xffffffffu, int(valid), 1) != 0;
+                    if (!valid) continue;
+                    const bool next = lane != 31 && nvalid && noff == off[u] + V;
+                    const bool prev = lane != 0 && poff + V == off[u];
+                    T* a = static_cast<T*>(dst) + off[u];
+                    if (next) {
+                        *reinterpret_cast<uint4*>(a - ph + V) = shift16(lo, hi, uint32_t((V - ph) * ES));
+                    } else {
+                        T e[V];
+                        memcpy(e, &val[u], sizeof e);
+#pragma unroll
+                        for (int k = 1; k < V; ++k)
+                            if (k >= V - ph) a[k] = e[k];
+                    }
+                    if (!prev) {
+                        T e[V];
+                        memcpy(e, &val[u], sizeof e);
+#pragma unroll
+                        for (int k = 0; k < V - 1; ++k)
+                            if (k < V - ph) a[k] = e[k];
+                    }
+                }
+                continue;
+            }
+        }
+#pragma unroll
+        for (int u = 0; u < kU; ++u)
+            if (v0 + 32 * u < v_end)
+                reinterpret_cast<VT*>(static_cast<T*>(dst) + (MODE == 0 ? g[u] : off[u]))[0] = val[u];
     }
+}
+
+template <int ES, int V, int MODE, int NDU>
+__global__ void __launch_bounds__(256) tiler_pieces_kernel(const __grid_constant__ PiecesDev pd,
+                                                           const void* __restrict__ src, void* __restrict__ dst) {
+    const int32_t c = int32_t(blockIdx.x);   // one chunk per CTA (a persistent chunk loop measured slower)
+    int pc = 0;
+    while (pc + 1 < pd.npieces && pd.chunk0[pc + 1] <= c) ++pc;
+    // the piece's walk constants in registers, padded to NDU dims with unit extents on the outside: the digit
+    // loop is then fully unrolled without loads (the walk's instruction count bounds this kernel)
+    int32_t L[NDU], AL[NDU], GS[NDU];
+    uint32_t M[NDU], S[NDU];
+#pragma unroll
+    for (int d = 0; d < NDU; ++d) {
+        const int e = d - (NDU - pd.nd);
+        L[d] = e >= 0 ? pd.len[pc][e] : 1;
+        M[d] = e >= 0 ? pd.mul[pc][e] : 0u;
+        S[d] = e >= 0 ? pd.shift[pc][e] : 0u;
+        AL[d] = e >= 0 ? pd.p_lin[e] : 0;
+        GS[d] = e >= 0 ? pd.p_gst[e] : 0;
+    }
+    const int32_t v_begin = (c - pd.chunk0[pc]) * kPieceChunk;
+    const int32_t v_end = min(pd.nvec[pc], v_begin + kPieceChunk);
+    // vector pieces and the scalar slivers in one launch (a second launch for the slivers cost ~8 us)
+    if (V > 1 && pd.vec[pc])
+        pieces_walk<ES, V, MODE, NDU>(L, M, S, AL, GS, v_begin, v_end, pd.abase[pc], pd.tbase[pc], pd.phase[pc],
+                                      src, dst);
+    else
+        pieces_walk<ES, 1, MODE, NDU>(L, M, S, AL, GS, v_begin, v_end, pd.abase[pc], pd.tbase[pc], 0, src, dst);
 }
 
 // One piece under construction: a sub-range per combined dim, a wrap flag per array dim.
@@ -1213,9 +1330,10 @@ struct PieceBox {
 };
 
 // Split the parent tiler into affine pieces; false if it does not have the structure above (or needs more than
-// kMaxPieces pieces, or would not fit 31-bit offsets).  pieces_vec / pieces_scalar: pieces whose walk can use
-// V-element vectors, and the rest.
-bool make_pieces(const TilerDev& td, int es, const void* arr, const void* tiles, int V, PiecesDev* pv, PiecesDev* ps) {
+// kMaxPieces pieces, or would not fit 31-bit offsets).  Each piece is marked for V-element vectors or not;
+// *vec_elems counts the elements of the vector pieces.
+bool make_pieces(const TilerDev& td, int es, int mode, const void* arr, const void* tiles, int V, PiecesDev* P,
+                 int64_t* vec_elems) {
     if (td.linear || !td.fast32 || td.array_elems >= (int64_t(1) << 31) || td.total >= (int64_t(1) << 31)) return false;
     const int nd = td.nd, ra = td.ra;
     std::vector<PieceBox> boxes(1);
@@ -1281,9 +1399,7 @@ bool make_pieces(const TilerDev& td, int es, const void* arr, const void* tiles,
         boxes.swap(next);
         if (boxes.size() > size_t(2 * kMaxPieces)) return false;
     }
-    // build the two piece tables
-    std::memset(pv, 0, sizeof *pv);
-    std::memset(ps, 0, sizeof *ps);
+    // build the piece table
     int64_t lin[2 * AOL_MAX_RANK], gst[2 * AOL_MAX_RANK];
     {
         int64_t g = 1;
@@ -1308,12 +1424,12 @@ bool make_pieces(const TilerDev& td, int es, const void* arr, const void* tiles,
         for (; pos < nd - 1; ++pos) order[pos] = order[pos + 1];
         order[nd - 1] = nd - 1;
     }
-    for (PiecesDev* P : {pv, ps}) {
-        P->nd = nd;
-        for (int i = 0; i < nd; ++i) {
-            P->p_lin[i] = int32_t(lin[order[i]]);
-            P->p_gst[i] = int32_t(gst[order[i]]);
-        }
+    std::memset(P, 0, sizeof *P);
+    *vec_elems = 0;
+    P->nd = nd;
+    for (int i = 0; i < nd; ++i) {
+        P->p_lin[i] = int32_t(lin[order[i]]);
+        P->p_gst[i] = int32_t(gst[order[i]]);
     }
     const uintptr_t ptrs = reinterpret_cast<uintptr_t>(arr) | reinterpret_cast<uintptr_t>(tiles);
     for (const PieceBox& b : boxes) {
@@ -1326,11 +1442,14 @@ bool make_pieces(const TilerDev& td, int es, const void* arr, const void* tiles,
         if (count == 0) continue;
         for (int a = 0; a < ra; ++a) ab += (td.org[a] - (((b.wrapped >> a) & 1) ? td.ashape[a] : 0)) * td.astride[a];
         // vectors: the innermost walked dim unit-stride on both sides, extents / bases / strides multiples of V
+        // (a piece may start misaligned on the array side: every vector of the piece then shares the phase
+        // ab mod V; gathers read, and scatters write, the aligned 16 bytes around each vector, exchanging the
+        // overlap with the neighbouring lanes; a gather's second aligned load stays inside the allocation because
+        // the array's rows are a multiple of V elements long)
         const int last = order[nd - 1];
-        bool vec = V > 1 && lin[last] == 1 && gst[last] == 1 && b.len[last] % V == 0 && ab % V == 0 && tb % V == 0 &&
-                   ptrs % uintptr_t(V * es) == 0;
+        bool vec = V > 1 && lin[last] == 1 && gst[last] == 1 && b.len[last] % V == 0 && tb % V == 0 &&
+                   ptrs % uintptr_t(V * es) == 0 && (ab % V == 0 || mode == 1 || td.ashape[ra - 1] % V == 0);
         for (int i = 0; i < nd - 1 && vec; ++i) vec = lin[order[i]] % V == 0 && gst[order[i]] % V == 0;
-        PiecesDev* P = vec ? pv : ps;
         if (P->npieces == kMaxPieces) return false;
         const int k = P->npieces++;
         for (int i = 0; i < nd; ++i) {
@@ -1340,13 +1459,30 @@ bool make_pieces(const TilerDev& td, int es, const void* arr, const void* tiles,
         P->abase[k] = int32_t(ab);
         P->tbase[k] = int32_t(tb);
         P->nvec[k] = int32_t(count / (vec ? V : 1));
+        P->phase[k] = vec ? int32_t(ab % V) : 0;
+        P->vec[k] = vec ? 1 : 0;
+        if (vec) *vec_elems += count;
     }
-    for (PiecesDev* P : {pv, ps}) {
-        P->chunk0[0] = 0;
-        for (int k = 0; k < P->npieces; ++k) P->chunk0[k + 1] = P->chunk0[k] + (P->nvec[k] + kPieceChunk - 1) / kPieceChunk;
-        P->nchunks = P->chunk0[P->npieces];
-    }
-    return true;
+    P->chunk0[0] = 0;
+    for (int k = 0; k < P->npieces; ++k) P->chunk0[k + 1] = P->chunk0[k] + (P->nvec[k] + kPieceChunk - 1) / kPieceChunk;
+    P->nchunks = P->chunk0[P->npieces];
+    return P->npieces > 0;
+}
+
+// The digit loop unrolled for the smallest of 4 / 5 / 6 / 8 / 16 dims that holds the tiler's (5: a blocking of
+// a stack of planes, as in d3).
+template <int ES, int V, int MODE>
+void launch_pieces(const PiecesDev& p, const void* src, void* dst, cudaStream_t s) {
+    if (p.nd <= 4)
+        tiler_pieces_kernel<ES, V, MODE, 4><<<p.nchunks, 256, 0, s>>>(p, src, dst);
+    else if (p.nd == 5)
+        tiler_pieces_kernel<ES, V, MODE, 5><<<p.nchunks, 256, 0, s>>>(p, src, dst);
+    else if (p.nd <= 6)
+        tiler_pieces_kernel<ES, V, MODE, 6><<<p.nchunks, 256, 0, s>>>(p, src, dst);
+    else if (p.nd <= 8)
+        tiler_pieces_kernel<ES, V, MODE, 8><<<p.nchunks, 256, 0, s>>>(p, src, dst);
+    else
+        tiler_pieces_kernel<ES, V, MODE, kND><<<p.nchunks, 256, 0, s>>>(p, src, dst);
 }
 
 // AOL_TILER_PIECES=0 disables the affine-piece path (A/B measurements only).
@@ -1630,35 +1766,28 @@ aol_status_t launch_v(const TilerDev& td, const void* src, void* dst, unsigned l
             return AOL_OK;
         }
         const int g32 = int(std::max<int64_t>(1, std::min<int64_t>((td.total / V + 255) / 256, int64_t(dev.num_sms) * 128)));
-        tiler_linear32_kernel<ES, V, MODE><<<g32, 256, 0, s>>>(td, src, dst);
+        if (td.nd <= 3)
+            tiler_linear32_kernel<ES, V, MODE, 3><<<g32, 256, 0, s>>>(td, src, dst);
+        else if (td.nd <= 5)
+            tiler_linear32_kernel<ES, V, MODE, 5><<<g32, 256, 0, s>>>(td, src, dst);
+        else if (td.nd <= 8)
+            tiler_linear32_kernel<ES, V, MODE, 8><<<g32, 256, 0, s>>>(td, src, dst);
+        else
+            tiler_linear32_kernel<ES, V, MODE, kND><<<g32, 256, 0, s>>>(td, src, dst);
         AOL_LAUNCH_CHECK("tiler_linear32_kernel");
         return AOL_OK;
     }
     if constexpr (V == 1) {
         if (MODE <= 1 && !lin && tiler_pieces_enabled()) {
             constexpr int VV = 16 / ES;
-            PiecesDev pv, ps;
+            PiecesDev pd;
+            int64_t nv = 0;
             // only when (nearly) all elements run as 16-byte vectors: scalar pieces lose to the box kernel
-            bool use = make_pieces(td, ES, MODE == 0 ? src : dst, MODE == 0 ? dst : src, VV, &pv, &ps);
+            const bool use = VV > 1 && make_pieces(td, ES, MODE, MODE == 0 ? src : dst, MODE == 0 ? dst : src, VV,
+                                                   &pd, &nv) && 10 * nv >= 9 * td.total;
             if (use) {
-                int64_t nv = 0;
-                for (int k = 0; k < pv.npieces; ++k) nv += int64_t(pv.nvec[k]) * VV;
-                use = 10 * nv >= 9 * td.total;
-            }
-            if (use) {
-                DeviceInfo dev;
-                aol_status_t st = device_info(&dev);
-                if (st != AOL_OK) return st;
-                if (pv.npieces > 0) {
-                    const int gp = int(std::max<int64_t>(1, std::min<int64_t>(pv.nchunks, int64_t(dev.num_sms) * 8)));
-                    if constexpr (VV > 1) tiler_pieces_kernel<ES, VV, MODE><<<gp, 256, 0, s>>>(pv, src, dst);
-                    AOL_LAUNCH_CHECK("tiler_pieces_kernel");
-                }
-                if (ps.npieces > 0) {
-                    const int gp = int(std::max<int64_t>(1, std::min<int64_t>(ps.nchunks, int64_t(dev.num_sms) * 8)));
-                    tiler_pieces_kernel<ES, 1, MODE><<<gp, 256, 0, s>>>(ps, src, dst);
-                    AOL_LAUNCH_CHECK("tiler_pieces_kernel");
-                }
+                if constexpr (VV > 1) launch_pieces<ES, VV, MODE>(pd, src, dst, s);
+                AOL_LAUNCH_CHECK("tiler_pieces_kernel");
                 return AOL_OK;
             }
         }

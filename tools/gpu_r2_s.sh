@@ -1,7 +1,7 @@
 #!/bin/bash
 cd "$GRAFT_REPO_ROOT"
 mkdir -p gpurun_out
-timeout 900 python -m pytest tests/test_gpu_tiler_box.py -q -x > gpurun_out/r2s_tests.log 2>&1
+timeout 900 python -m pytest tests/test_gpu_tiler_box.py -q > gpurun_out/r2s_tests.log 2>&1
 echo "tests rc=$?" >> gpurun_out/r2s_tests.log
 timeout 900 python -m pytest tests/test_gpu_parity.py -q -x -k tiler >> gpurun_out/r2s_tests.log 2>&1
 echo "tests2 rc=$?" >> gpurun_out/r2s_tests.log
