@@ -1155,18 +1155,24 @@ struct PiecesDev {
 };
 
 // 16 bytes starting `b` bytes (0..15) into the 32 bytes (lo, hi): the misaligned array-side read of a vector
-// whose aligned neighbours were loaded instead (funnel shifts; b is uniform across the warp).
+// whose aligned neighbours were loaded instead (funnel shifts; b is uniform across the CTA, so the word offset is a
+// uniform branch rather than a select chain per word).
 __device__ __forceinline__ uint4 shift16(const uint4& lo, const uint4& hi, uint32_t b) {
-    const uint32_t w[8] = {lo.x, lo.y, lo.z, lo.w, hi.x, hi.y, hi.z, hi.w};
-    const uint32_t wb = b >> 2, sh = (b & 3u) * 8u;
-    uint32_t r[4];
-#pragma unroll
-    for (int q = 0; q < 4; ++q) {
-        const uint32_t a0 = wb == 0 ? w[q] : wb == 1 ? w[q + 1] : wb == 2 ? w[q + 2] : w[q + 3];
-        const uint32_t a1 = wb == 0 ? w[q + 1] : wb == 1 ? w[q + 2] : wb == 2 ? w[q + 3] : w[q + 4];
-        r[q] = __funnelshift_r(a0, a1, sh);
+    const uint32_t sh = (b & 3u) * 8u;
+    switch (b >> 2) {
+        case 0:
+            return make_uint4(__funnelshift_r(lo.x, lo.y, sh), __funnelshift_r(lo.y, lo.z, sh),
+                              __funnelshift_r(lo.z, lo.w, sh), __funnelshift_r(lo.w, hi.x, sh));
+        case 1:
+            return make_uint4(__funnelshift_r(lo.y, lo.z, sh), __funnelshift_r(lo.z, lo.w, sh),
+                              __funnelshift_r(lo.w, hi.x, sh), __funnelshift_r(hi.x, hi.y, sh));
+        case 2:
+            return make_uint4(__funnelshift_r(lo.z, lo.w, sh), __funnelshift_r(lo.w, hi.x, sh),
+                              __funnelshift_r(hi.x, hi.y, sh), __funnelshift_r(hi.y, hi.z, sh));
+        default:
+            return make_uint4(__funnelshift_r(lo.w, hi.x, sh), __funnelshift_r(hi.x, hi.y, sh),
+                              __funnelshift_r(hi.y, hi.z, sh), __funnelshift_r(hi.z, hi.w, sh));
     }
-    return make_uint4(r[0], r[1], r[2], r[3]);
 }
 
 // The walk of one chunk of a piece with W-element accesses (W = the vector width, or 1 for a piece that cannot
