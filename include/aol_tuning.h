@@ -21,6 +21,9 @@
 #define AOL_FLAG_ROW_STAGES 512     /* int32 input: one row per TMA ring stage (default when a row triple
                                        exceeds a third of the ring's bytes: W > 3271)                        */
 #define AOL_FLAG_TRIPLE_STAGES 1024 /* int32 input: one row triple per ring stage for any W                  */
+#define AOL_FLAG_I32_STRIPS 2048    /* int32 input, W % 32 == 0: column strips of ~64 repetitions (default:
+                                       strips of <= 512 only when W / 8 exceeds one CTA's 992 consumers, i.e.
+                                       W > 7936; lets the tests exercise several strips at small widths)     */
 
 #ifdef __cplusplus
 extern "C" {

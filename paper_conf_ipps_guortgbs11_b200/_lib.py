@@ -60,9 +60,9 @@ class aol_filter_t(ctypes.Structure):
 
 # aol_launch_opts_t.flags bits (include/aol_tuning.h AOL_FLAG_*; A/B experiments, results are identical)
 FLAG_U8_ONE_REP, FLAG_NO_PDL, FLAG_I32_LINEAR = 32, 64, 128
-FLAG_ROW_STAGES, FLAG_TRIPLE_STAGES = 512, 1024
+FLAG_ROW_STAGES, FLAG_TRIPLE_STAGES, FLAG_I32_STRIPS = 512, 1024, 2048
 FLAGS = {"U8_ONE_REP": FLAG_U8_ONE_REP, "NO_PDL": FLAG_NO_PDL, "I32_LINEAR": FLAG_I32_LINEAR,
-         "ROW_STAGES": FLAG_ROW_STAGES, "TRIPLE_STAGES": FLAG_TRIPLE_STAGES}
+         "ROW_STAGES": FLAG_ROW_STAGES, "TRIPLE_STAGES": FLAG_TRIPLE_STAGES, "I32_STRIPS": FLAG_I32_STRIPS}
 
 
 class aol_launch_opts_t(ctypes.Structure):

@@ -346,7 +346,7 @@ aol_status_t check_frame_args(const void* d_in, aol_dtype_t in_dtype, const void
 }
 
 constexpr int32_t kKnownFlags = AOL_FLAG_U8_ONE_REP | AOL_FLAG_NO_PDL | AOL_FLAG_I32_LINEAR | AOL_FLAG_ROW_STAGES |
-                                AOL_FLAG_TRIPLE_STAGES;
+                                AOL_FLAG_TRIPLE_STAGES | AOL_FLAG_I32_STRIPS;
 
 aol_status_t check_opts(const aol_launch_opts_t* opts) {
     if (opts && (opts->ctas_per_sm < 0 || opts->ctas_per_sm > 8 || opts->stages < 0 || opts->bands_per_unit < 0 ||

@@ -53,24 +53,46 @@ aol_status_t get_encode_fn(EncodeTiledFn* fn) {
     return AOL_OK;
 }
 
+// Column strips (int32, W % 32 == 0): repetitions per strip, a multiple of 32 (0: no strips).  Frames wider than
+// one CTA's 992 consumer threads (W > 7936) run as strips of <= 480 repetitions (8K DCI: 352 + 352 + 320); the
+// strips of a row are balanced.  AOL_FLAG_I32_STRIPS forces ~64-repetition strips (tests: several strips at small widths).
+int i32_strip_reps(aol_dtype_t dt, int64_t W, int flags) {
+    if (dt != AOL_I32 || W % 32 != 0) return 0;
+    const int64_t reps = W / 8;
+    static const int per_env = [] {   // AOL_STRIP_REPS=n: strips of <= n repetitions (A/B measurements only)
+        const char* e = std::getenv("AOL_STRIP_REPS");
+        return e ? std::max(32, std::min(kMaxConsumers, std::atoi(e))) : 0;
+    }();
+    int64_t per = 0;
+    if (flags & AOL_FLAG_I32_STRIPS)
+        per = 64;
+    else if (reps > kMaxConsumers)
+        per = per_env > 0 ? per_env : 480;   // <= 512 threads per CTA: the 64-register 1024-thread build spills
+    else
+        return 0;
+    const int64_t n = (reps + per - 1) / per;
+    return int(((reps + n - 1) / n + 31) / 32 * 32);
+}
+
 // Shared-memory layout of an int32 row triple (the kernel's kSwz): 128 = TMA tensor loads of 128-byte lines
 // under SWIZZLE_128B (W % 32 == 0); 0 = one 1-D bulk copy of the contiguous triple into linear rows (W % 32 != 0,
-// or forced by AOL_FLAG_I32_LINEAR).  -1 for uint8 input.
+// or forced by AOL_FLAG_I32_LINEAR); 1 = column strips (i32_strip_reps), one row per stage.  -1 for uint8 input.
 int i32_layout(aol_dtype_t dt, int64_t W, int flags) {
     if (dt != AOL_I32) return -1;
+    if (i32_strip_reps(dt, W, flags) > 0) return 1;
     if (flags & AOL_FLAG_I32_LINEAR) return 0;
     return W % 32 == 0 ? 128 : 0;
 }
 
 bool tma_shape_ok(aol_dtype_t dt, int64_t planes, int64_t channels, int64_t H, int64_t W, int flags) {
-    if (H < 9 || W / 8 > kMaxConsumers) return false;
+    if (H < 9 || (W / 8 > kMaxConsumers && i32_layout(dt, W, flags) != 1)) return false;
     // checksum weights (1 + frame-local output index) are computed in 32 bits
     if (channels * (4 * (H / 9)) * (3 * (W / 8)) >= (int64_t(1) << 32) - 1) return false;
     // int32 tensor layout: {32, W/32, 3}-element boxes under SWIZZLE_128B (a box dimension holds at most 256
     // elements; tensor row coordinates are int32); linear rows: 1-D bulk copies of 12W bytes (16-byte multiple
     // since W % 8 == 0)
     if (dt == AOL_I32) {
-        if (i32_layout(dt, W, flags) == 0) return true;
+        if (i32_layout(dt, W, flags) <= 1) return true;   // 1-D bulk copies
         return W / 32 <= 256 && planes * H < (int64_t(1) << 31);
     }
     if (dt == AOL_U8) return W % 16 == 0;   // 1-D bulk copies: 16-byte granularity
@@ -88,6 +110,7 @@ KernelFn pick(aol_dtype_t dt, int out_es, bool checksum, int kr, int64_t W, int 
 // bytes the ring keeps in flight (4K: 46 KB triples vs 115 KB per SM), unless forced by a flag.
 int rows_per_stage(aol_dtype_t dt, int64_t W, int flags) {
     if (dt != AOL_I32) return 3;
+    if (i32_layout(dt, W, flags) == 1) return 1;   // column strips: one row (of the strip) per stage
     if (flags & AOL_FLAG_ROW_STAGES) return 1;
     if (flags & AOL_FLAG_TRIPLE_STAGES) return 3;
     return 12 * W > kInflightBytesPerSM / 3 ? 1 : 3;
@@ -108,6 +131,11 @@ RingGeom ring_geom(aol_dtype_t dt, int out_es, int64_t W, int flags) {
     g.stage_bytes = uint32_t(rows_per_stage(dt, W, flags) * W) * es;
     g.stage_stride = (g.stage_bytes + align - 1) & ~(align - 1);
     g.out_bytes = uint32_t(4 * out_es * (3 * (W / 8))) * (dt == AOL_RGB8 ? 3u : 1u);   // packed: 3 planes
+    if (const int sr = i32_strip_reps(dt, W, flags)) {   // a strip row + the next repetition's first 16 bytes
+        g.stage_bytes = uint32_t(32 * sr + 16);
+        g.stage_stride = (g.stage_bytes + align - 1) & ~(align - 1);
+        g.out_bytes = uint32_t(4 * out_es * 3 * sr);
+    }
     return g;
 }
 
@@ -193,7 +221,9 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void*
     // 1 for narrower ones (CIF: 0.361 vs 0.315 ms -- one half-idle warp per CTA) and for int32
     // (profiles/r01_u8_r2_ab.jsonl)
     const int kr = rgb ? 3 : (in_dtype == AOL_U8 && W >= 1024 && !(o.flags & AOL_FLAG_U8_ONE_REP)) ? 2 : 1;
-    const int nc = int(((W / 8 / (rgb ? 1 : kr)) + 31) / 32 * 32);   // packed: one repetition (3 channels) per thread
+    const int strip = i32_strip_reps(in_dtype, W, o.flags);   // column strips: consumers = repetitions per strip
+    const int64_t nstrips = strip > 0 ? (W / 8 + strip - 1) / strip : 1;
+    const int nc = strip > 0 ? strip : int(((W / 8 / (rgb ? 1 : kr)) + 31) / 32 * 32);   // packed: one repetition (3 channels) per thread
     const int block = nc + 32;
     int stages = 0, cps = 1;
     if (tma_ok) {
@@ -237,8 +267,8 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void*
     }
     if (o.kernel == 1 && !tma_ok) {
         set_error("TMA fused kernel requested but unsupported for this shape/dtype/alignment "
-                  "(W <= 7936 and a 2-stage ring within shared memory; uint8: W %% 16 == 0; 16-byte aligned "
-                  "buffers)");
+                  "(W <= 7936, or int32 with W %% 32 == 0 (column strips), and a 2-stage ring within shared memory; "
+                  "uint8: W %% 16 == 0; 16-byte aligned buffers)");
         return AOL_E_SHAPE;
     }
     if (o.kernel == 2) tma_ok = false;
@@ -270,7 +300,7 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void*
             double cost[kMaxNb + 1] = {};
             double best = 1e300;
             for (int cand = 1; cand <= max_nb; ++cand) {
-                const int64_t units = planes * ((nbands + cand - 1) / cand);
+                const int64_t units = planes * nstrips * ((nbands + cand - 1) / cand);
                 const int64_t waves = (units + max_ctas - 1) / max_ctas;
                 cost[cand] = double(waves) * (3.0 * cand + 1.0 + ovh);
                 best = std::min(best, cost[cand]);
@@ -287,7 +317,7 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void*
         nb = std::max(1, std::min(nb, nbands));
         plan->kernel = 1;
         plan->bands_per_unit = nb;
-        plan->units_per_plane = (nbands + nb - 1) / nb;
+        plan->units_per_plane = int(nstrips * ((nbands + nb - 1) / nb));
         plan->units = planes * plan->units_per_plane;
         plan->grid = int(std::min<int64_t>(plan->units, max_ctas));
         plan->block = block;
@@ -317,7 +347,7 @@ aol_status_t prepare_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t 
     std::memset(&L->map, 0, sizeof L->map);
     const bool u8_tensor = in_dtype == AOL_U8 && W % 128 == 0 && W / 128 <= 256 && planes * H < (int64_t(1) << 31);
     const int layout = i32_layout(in_dtype, W, plan.flags);
-    if (layout > 0 || u8_tensor) {
+    if (layout == 128 || u8_tensor) {
         aol_status_t st = encode_row_map(&L->map, in_dtype, d_in, planes * H, W, plan.flags);
         if (st != AOL_OK) return st;
     }
@@ -343,6 +373,7 @@ aol_status_t prepare_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t 
     a.row_pitch = int32_t(rgb ? 3 * W : W);
     a.reps = int32_t(W / 8);
     a.segs = int32_t(W / 32);   // int32 swizzled 128-byte lines per row (unused for linear rows)
+    if (layout == 1) a.segs = i32_strip_reps(in_dtype, W, plan.flags);   // column strips: repetitions per strip
     a.triples_per_plane = int32_t(H / 3);
     a.nbands = int32_t(H / 9);
     a.bands_per_unit = plan.bands_per_unit;

@@ -7,6 +7,8 @@ KernelFn tma_kernel_i32_cs(int block, int cps);
 KernelFn tma_kernel_i32_nocs(int block, int cps);
 KernelFn tma_kernel_i32l_cs(int block, int cps);
 KernelFn tma_kernel_i32l_nocs(int block, int cps);
+KernelFn tma_kernel_i32s_cs(int block, int cps);
+KernelFn tma_kernel_i32s_nocs(int block, int cps);
 KernelFn tma_kernel_u8_cs(int block, int cps);
 KernelFn tma_kernel_u8_nocs(int block, int cps);
 KernelFn tma_kernel_u8r2_cs(int block, int cps);
@@ -28,6 +30,7 @@ KernelFn tma_kernel_rgb8(bool checksum, bool out16, int block, int cps) {
 
 KernelFn tma_kernel_i32(bool checksum, int layout, int block, int cps) {
     if (layout == 0) return checksum ? tma_kernel_i32l_cs(block, cps) : tma_kernel_i32l_nocs(block, cps);
+    if (layout == 1) return checksum ? tma_kernel_i32s_cs(block, cps) : tma_kernel_i32s_nocs(block, cps);
     return checksum ? tma_kernel_i32_cs(block, cps) : tma_kernel_i32_nocs(block, cps);
 }
 KernelFn tma_kernel_u8(bool checksum, bool out16, int reps_per_thread, int block, int cps) {

@@ -150,7 +150,7 @@ __device__ __forceinline__ void h_row(uint32_t row_base, uint32_t rr, const RepG
         static_assert(kR == 1, "int32 path: one repetition per thread");
         const uint32_t line = rr * segs + g.seg;
         int4 q0, q1;
-        if constexpr (kSwz == 0) {
+        if constexpr (kSwz == 0 || kSwz == 1) {
             // linear rows (1-D bulk copies): a thread's 32 bytes sit at 32r, so a quarter-warp's first loads
             // would hit each 16-byte bank group twice; lanes with bit 2 set load their upper chunk first,
             // which spreads every quarter-warp's 8 chunks over all 8 bank groups (conflict-free LDS.128)
@@ -171,7 +171,7 @@ __device__ __forceinline__ void h_row(uint32_t row_base, uint32_t rr, const RepG
         const int32_t qp = q + p;
         int32_t dn = __shfl_down_sync(0xffffffffu, d, 1);
         int4 qn = q0;   // lane 31 / wrapping repetition: neighbour chunk from smem (predicated, no branch)
-        if constexpr (kSwz == 0)
+        if constexpr (kSwz == 0 || kSwz == 1)
             ptx::lds128_if(qn, row_base + rr * (4u * W) + g.offn, g.fix);
         else
             ptx::lds128_if(qn, row_base + swz(rr * segs + g.segn, g.offn), g.fix);
@@ -257,7 +257,11 @@ __device__ __forceinline__ void h_row(uint32_t row_base, uint32_t rr, const RepG
 // 8 columns); 1 or 2 for uint8 input, whose 16 bytes for two repetitions come in one LDS.128 and whose per-stage
 // bookkeeping (mbarrier wait/arrive, addressing) two repetitions then share (the host picks, fused.cu).
 // kSwz = the int32 smem layout: 128 (TMA tensor loads under SWIZZLE_128B, W % 32 == 0) or 0 (1-D bulk copies,
-// linear rows, any W % 8 == 0; the default when W % 32 != 0); 3 = packed 24-bit pixels; 0 for planar uint8.
+// linear rows, any W % 8 == 0; the default when W % 32 != 0) or 1 (column strips for frames wider than one CTA's
+// 992 consumer threads, W % 32 == 0: a unit is (plane, strip of a.segs repetitions, run of bands); a stage is
+// one row of the strip, 1-D bulk copies of the strip's 32 bytes per repetition plus 16 bytes of the next
+// repetition -- the row-wrapping strip's from column 0 -- into linear rows; each band's 4 output rows leave as
+// 4 row-segment bulk stores); 3 = packed 24-bit pixels; 0 for planar uint8.
 // (SWIZZLE_32B tensor lines for W % 32 != 0 measured no faster than linear rows and were removed,
 // profiles/r01_i32_layout_ab.jsonl.)  Tout = output element: int32, or int16 for 8-bit samples ([-5, 255]).
 template <typename Tin, typename Tout, int kR, int kSwz, bool kChecksum, int kMaxThreads, int kMinBlocks>
@@ -265,6 +269,7 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
     fused_tma_kernel(const __grid_constant__ CUtensorMap tmap, const FusedArgs a) {
     constexpr bool kI32 = std::is_same<Tin, int32_t>::value;
     constexpr bool kIL = !kI32 && kSwz == 3;   // packed 24-bit pixels: a unit covers the 3 planes of a frame
+    constexpr bool kStrip = kI32 && kSwz == 1; // column strips (a.segs repetitions each, one row per stage)
     constexpr int kC = 3 * kR;                 // Y / Z columns per consumer thread (kIL: 3 channels x 3)
     constexpr int kRP = kIL ? 1 : kR;          // H-tiler repetitions per consumer thread
     extern __shared__ uint8_t smem_raw[];
@@ -297,7 +302,16 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
             uint32_t ph = 0;
             for (int64_t k = 0, u = unit_of(a, 0); u < a.nunits; u = unit_of(a, ++k)) {
                 const int64_t plane = u / a.units_per_plane;
-                const int32_t b0 = int32_t(u - plane * a.units_per_plane) * a.bands_per_unit;
+                int32_t run = int32_t(u - plane * a.units_per_plane), rs0 = 0, rs1 = a.reps;
+                if constexpr (kStrip) {   // unit = (plane, strip, run of bands), runs innermost
+                    const int32_t nstrips = (a.reps + a.segs - 1) / a.segs;
+                    const int32_t runs = a.units_per_plane / nstrips;
+                    const int32_t strip = run / runs;
+                    run -= strip * runs;
+                    rs0 = strip * a.segs;
+                    rs1 = min(rs0 + a.segs, a.reps);
+                }
+                const int32_t b0 = run * a.bands_per_unit;
                 const int32_t b1 = min(b0 + a.bands_per_unit, a.nbands);
                 const int32_t ntrip = 3 * (b1 - b0) + 1;
                 const int64_t row0 = plane * a.H;
@@ -309,9 +323,24 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
                         if (a.rows_per_stage == 1) {   // one row per stage, three stages per triple
                             for (int32_t q = 0; q < 3; ++q) {
                                 ptx::mbar_wait_sleep(&empty[s], ph ^ 1u);
-                                ptx::mbar_arrive_expect_tx(&full[s], a.stage_bytes);
                                 uint8_t* dst = stage_base + size_t(s) * a.stage_stride;
                                 const int64_t row = row0 + 3 * trip + q;
+                                if constexpr (kStrip) {
+                                    // the strip's repetitions, then the next repetition's first 16 bytes (its
+                                    // first 3 columns are the last pattern overlap; column 0 for the last strip)
+                                    const uint32_t main = 32u * uint32_t(rs1 - rs0);
+                                    const uint8_t* xr = static_cast<const uint8_t*>(a.X) + size_t(row) * 4u * a.W;
+                                    ptx::mbar_arrive_expect_tx(&full[s], main + 16u);
+                                    ptx::bulk_load(dst, xr + 32u * uint32_t(rs0), main, &full[s]);
+                                    ptx::bulk_load(dst + main, xr + (rs1 == a.reps ? 0u : 32u * uint32_t(rs1)), 16u,
+                                                   &full[s]);
+                                    if (++s == a.stages) {
+                                        s = 0;
+                                        ph ^= 1u;
+                                    }
+                                    continue;
+                                }
+                                ptx::mbar_arrive_expect_tx(&full[s], a.stage_bytes);
                                 if constexpr (kSwz == 0)
                                     ptx::bulk_load(dst, static_cast<const uint8_t*>(a.X) + size_t(row) * 4u * a.W,
                                                    a.stage_bytes, &full[s]);
@@ -353,8 +382,8 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
 
     // ---------------------------------------------------- consumer threads
     const int lane = tid & 31;
-    const bool active = kRP * tid < a.reps;
-    const int r = active ? kRP * tid : a.reps - kRP;   // first repetition owned (clamped for idle lanes)
+    bool active = kRP * tid < a.reps;
+    int r = active ? kRP * tid : a.reps - kRP;   // first repetition owned (clamped for idle lanes)
     const int rn = (r + kRP == a.reps) ? 0 : r + kRP;  // next thread's repetition (toroidal, Fig. 11 '% 1920')
     RepGeom g;
     g.fix = (lane == 31) || (r + 1 == a.reps);
@@ -387,6 +416,7 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
     const uint32_t segs = uint32_t(a.segs);
     const uint32_t Wu = uint32_t(a.W);
     const int Wo = a.Wo;
+    int ow = Wo, rl = r;   // output staging: row pitch (elements) and the thread's repetition within it
     const uint32_t stage_s32 = ptx::smem_u32(stage_base);
 
     int s = 0;
@@ -395,7 +425,26 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
 
     for (int64_t k = 0, u = unit_of(a, 0); u < a.nunits; u = unit_of(a, ++k)) {
         const int64_t plane = u / a.units_per_plane;
-        const int32_t b0 = int32_t(u - plane * a.units_per_plane) * a.bands_per_unit;
+        int32_t run = int32_t(u - plane * a.units_per_plane), rs0 = 0;
+        if constexpr (kStrip) {   // this unit's strip: repetitions rs0 .. rs0 + nr - 1, rows of 32 nr + 16 bytes
+            const int32_t nstrips = (a.reps + a.segs - 1) / a.segs;
+            const int32_t runs = a.units_per_plane / nstrips;
+            const int32_t strip = run / runs;
+            run -= strip * runs;
+            rs0 = strip * a.segs;
+            const int32_t nr = min(a.segs, a.reps - rs0);
+            active = tid < nr;
+            rl = active ? tid : nr - 1;
+            r = rs0 + rl;
+            ow = 3 * nr;
+            g.seg = g.segn = 0;
+            g.swap = ((lane >> 2) & 1) != 0;   // as kSwz = 0 (rs0 is a multiple of 32)
+            g.off0 = 32u * uint32_t(rl) + (g.swap ? 16u : 0u);
+            g.off1 = 32u * uint32_t(rl) + (g.swap ? 0u : 16u);
+            g.offn = 32u * uint32_t(rl + 1);   // the last thread: the 16 bytes after the strip
+            g.fix = (lane == 31) || (rl + 1 == nr);
+        }
+        const int32_t b0 = run * a.bands_per_unit;
         const int32_t b1 = min(b0 + a.bands_per_unit, a.nbands);
         const int32_t chan = int32_t(plane % a.channels);
         uint64_t csacc = 0;
@@ -445,7 +494,7 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
             } else if (active) {
 #pragma unroll
                 for (int k = 0; k < 4; ++k) {
-                    const uint32_t e0 = uint32_t(k * Wo + 3 * r);   // element index of the thread's first column
+                    const uint32_t e0 = uint32_t(k * ow + 3 * rl);   // element index of the thread's first column
                     if constexpr (sizeof(Tout) == 4 && kR == 1) {
 #pragma unroll
                         for (int m = 0; m < 3; ++m) ptx::sts32(ob + 4u * (e0 + m), z[k][m]);
@@ -472,6 +521,13 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
                     Tout* gz = static_cast<Tout*>(a.Z) + (size_t(3 * plane + j) * a.Ho + size_t(4 * band)) * size_t(Wo);
                     ptx::bulk_store(gz, outbuf + (emit_idx % kOutBufs) * a.out_bytes + j * pb, pb);
                 }
+                ptx::bulk_commit();
+            } else if (kStrip && tid == 0) {   // 4 row segments of the strip
+                Tout* gz = static_cast<Tout*>(a.Z) + (size_t(plane) * a.Ho + size_t(4 * band)) * size_t(Wo) + 3 * rs0;
+                const uint8_t* src = outbuf + (emit_idx % kOutBufs) * a.out_bytes;
+#pragma unroll
+                for (int k = 0; k < 4; ++k)
+                    ptx::bulk_store(gz + size_t(k) * Wo, src + k * ow * int(sizeof(Tout)), uint32_t(ow * sizeof(Tout)));
                 ptx::bulk_commit();
             } else if (tid == 0) {
                 Tout* gz = static_cast<Tout*>(a.Z) + (size_t(plane) * a.Ho + size_t(4 * band)) * size_t(Wo);
@@ -705,7 +761,7 @@ struct FusedLaunch {
 };
 
 // Explicit instantiations live in fused_k_*.cu (compiled in parallel); these pick one.
-KernelFn tma_kernel_i32(bool checksum, int layout, int block, int cps);   // layout = kSwz (128 or 0)
+KernelFn tma_kernel_i32(bool checksum, int layout, int block, int cps);   // layout = kSwz (128, 0 or 1)
 KernelFn tma_kernel_u8(bool checksum, bool out16, int reps_per_thread, int block, int cps);
 KernelFn tma_kernel_rgb8(bool checksum, bool out16, int block, int cps);   // packed 24-bit pixels
 
