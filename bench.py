@@ -24,7 +24,8 @@ in-run oracle parity flag: d1 (one HD frame: warm / cold-L2 / graph latency and
 host enqueue), d3 (generic tiler gather / FAST / SEQUENTIAL scatter on the
 SURVEY instance, a wrapping variant and the paper's H input tiler), d4 (64 4K
 frames), d5 (the 10,000-frame stream frame-sharded over the N ranks: strong
-scaling, at every N; every stream frame's checksum verified).
+scaling, at every N; every stream frame's checksum verified), wide (16 8K DCI
+frames, 8192 wide: the fused kernel's column strips).
 
 The cpu_baseline leg (N = 1, rank 0) times the CPU oracle (oracle/, test
 infrastructure) over ALL 300 frames of the d2 workload, reports frames/s and
@@ -50,7 +51,7 @@ if ROOT not in sys.path:
 
 METRIC = "HD->SD downscale frames/sec (1/2/4/8 B200) and achieved HBM GB/s vs peak"
 FALLBACK_HBM_GBS = 6650.0  # /opt/skills/guides/B200_PROFILING.md fallback
-ALL_EXTRAS = ("d1", "d3", "d4", "d5")
+ALL_EXTRAS = ("d1", "d3", "d4", "d5", "wide")
 
 
 def parse(argv=None):
@@ -605,6 +606,35 @@ def record_d4(aol, peak, check):
     return rec
 
 
+def record_wide(aol, peak, check):
+    """Frames wider than one CTA's consumer threads: 16 8K DCI frames (4320 x 8192 x 3, int32) through the fused
+    kernel's column strips (W > 7936); all 16 checksums against the oracle."""
+    import numpy as np
+    import torch
+
+    N, C, H, W, seed = 16, 3, 4320, 8192, 2
+    x = aol.synth_frames(seed, 0, N, C, H, W)
+    z = torch.empty((N, C, 4 * (H // 9), 3 * (W // 8)), dtype=torch.int32, device="cuda")
+    cs = torch.empty(N, dtype=torch.uint64, device="cuda")
+    med, mn = timed(lambda: aol.downscale_frame(x, out=z, checksums=cs), inner=5)
+    b = N * frame_bytes(C, H, W)
+    rec = {"config": "16 8K DCI frames 8192x4320x3 int32 -> 3072x1920 (column strips: W > 7936)", "ms": med,
+           "min_ms": mn, "frames_per_s": N / (med / 1e3), "GBps": b / med / 1e6, "frac": b / med / 1e6 / peak,
+           "kernel": aol.last_kernel(), "timing": "CUDA events, 5 calls back to back per event pair, median of 20",
+           "plan": aol.downscale_frame_plan(N, C, H, W)}
+    torch.cuda.synchronize()
+    got = cs.cpu().view(torch.int64).numpy().view(np.uint64)
+    del x, z, cs
+    torch.cuda.empty_cache()
+    if check:
+        # 6 frames (18 planes for the oracle's plane-parallel threads, 2.5 GB of host buffer) at a time
+        ref, spent = oracle_checksums(seed, range(N), C, H, W, oracle_threads(), chunk=6)
+        rec["parity"] = bool(np.array_equal(ref, got))
+        rec["parity_scope"] = f"all {N} frame checksums vs the oracle"
+        rec["cpu_oracle_frames_per_s"] = N / spent
+    return rec
+
+
 def record_d5(a, aol, world, rank, use_dist, backend, d2_fps_per_gpu, peak, check):
     """configs[4]: the 10,000-frame HD stream frame-sharded across the ranks (strong scaling).
     Rank g owns stream frames [g*T/G, (g+1)*T/G) and cycles them through a device pool of 256 unique frames:
@@ -885,6 +915,8 @@ def main():
             records["d3"] = record_d3(aol, peak, check)
         if "d4" in extras:
             records["d4"] = record_d4(aol, peak, check)
+        if "wide" in extras:
+            records["wide"] = record_wide(aol, peak, check)
     if use_dist:
         dist.barrier()
 
