@@ -802,10 +802,13 @@ aol_status_t aol_filter_chain_apply(const aol_filter_t* f1, const aol_filter_t* 
     for (int a = 0; a < f1->out.array_rank; ++a)
         if (f1->out.array_shape[a] != f2->in.array_shape[a])
             return fail(AOL_E_SHAPE, "f1's output array is not f2's input array");
+    const bool unfused = std::getenv("AOL_CHAIN_UNFUSED") != nullptr;
+    // a row filter followed by a column filter (the paper's H -> V shape, any parameters): chain_sep.cu
+    if (!unfused && launch_sep_chain(f1, f2, d_in, d_out, s, &st)) return st;
     ChainDev cd;
     int smem = 0;
     const char* why = "";
-    const bool fused = std::getenv("AOL_CHAIN_UNFUSED") == nullptr && plan_chain(f1, f2, &cd, &smem, &why);
+    const bool fused = !unfused && plan_chain(f1, f2, &cd, &smem, &why);
     if (!fused) {
         // two launches through the caller's workspace (the intermediate array)
         const size_t need = size_t(prod(f1->out.array_shape, f1->out.array_rank)) * 4;

@@ -85,6 +85,11 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void*
 aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t in_dtype, void* d_out,
                           int64_t frames, int64_t channels, int64_t H, int64_t W, uint64_t* d_cs, cudaStream_t s);
 
+// chain_sep.cu: aol_filter_chain_apply's separable case (a row filter then a column filter).  false: not that
+// case (nothing done); true: handled, *st = the outcome.
+bool launch_sep_chain(const aol_filter_t* f1, const aol_filter_t* f2, const int32_t* d_in, int32_t* d_out,
+                      cudaStream_t s, aol_status_t* st);
+
 aol_status_t launch_downscale_h(const int32_t* d_in, int32_t* d_out, int64_t planes, int64_t H, int64_t W,
                                 cudaStream_t s);
 aol_status_t launch_downscale_v(const int32_t* d_in, int32_t* d_out, int64_t planes, int64_t H, int64_t W,

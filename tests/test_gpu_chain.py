@@ -1,6 +1,8 @@
 """f3 fused: two run-time repetitions chained in one kernel (aol_filter_chain_apply) against the oracle --
-the paper's H then V filters (= the fused downscaler), the reverse order, random chains with random
-windows and divisors, and the two-launch fallback through a workspace for chains that do not qualify."""
+the paper's H then V filters (= the fused downscaler; a row filter then a column filter: the separable chain
+kernel), random separable chains (any pattern lengths, paving steps, wrapping origins, windows, divisors, lead
+dims), the reverse order and random general chains (the general chain kernel), and the two-launch fallback
+through a workspace for chains that do not qualify."""
 import numpy as np
 import pytest
 import torch
@@ -29,7 +31,7 @@ def test_chain_h_then_v_equals_fused_downscaler(orc, shape):
     fv = aol.filter_preset(aol.FILTER_V, P, H, 3 * W // 8)
     z = aol.filter_chain_apply(fh, fv, x)
     torch.cuda.synchronize()
-    assert aol.last_kernel() == "chain_kernel"
+    assert aol.last_kernel() == "sep_chain_kernel"
     zf, _ = aol.downscale_frame(x.unsqueeze(1))
     assert torch.equal(z, zf[:, 0])
     if H * W <= 1080 * 1920:
@@ -109,7 +111,64 @@ def test_random_chains(orc, seed):
     out = torch.from_numpy(bg.copy()).cuda()
     aol.filter_chain_apply(f1, f2, torch.from_numpy(xh).cuda(), out=out)
     torch.cuda.synchronize()
-    assert aol.last_kernel() == "chain_kernel"
+    assert aol.last_kernel() in ("chain_kernel", "sep_chain_kernel")
+    assert np.array_equal(out.cpu().numpy(), want)
+
+
+def _eye(n, diag):
+    return [[(diag[a] if a == j else 0) for j in range(n)] for a in range(n)]
+
+
+@pytest.mark.parametrize("seed", range(48))
+def test_random_separable_chains(orc, seed):
+    """A row filter then a column filter with every parameter random: lead dims (planes), pattern lengths <= 16,
+    paving steps (patterns overlapping, abutting or leaving gaps along the row; p2 <= L2 down the columns),
+    origins wrapping the row several times and shifting the rows, 1-8 windows, divisors of either sign, column
+    origins on and off the 16-byte grid.  Expected: the oracle's gather -> C task -> scatter, twice."""
+    rng = np.random.default_rng(7700 + seed)
+    n = int(rng.integers(2, 5))
+    lead = [int(rng.integers(1, 4)) for _ in range(n - 2)]
+    HX, WX = int(rng.integers(1, 40)), int(rng.integers(4, 300))
+    if seed % 3 == 0:
+        WX = 4 * int(rng.integers(1, 75))
+
+    def windows(L):
+        ln = int(rng.integers(1, L + 1))
+        nw = int(rng.integers(1, 9))
+        return nw, ln, [int(rng.integers(0, L - ln + 1)) for _ in range(nw)], int(rng.choice([1, 2, 3, 6, 7, -1, -6, 100]))
+
+    L1 = int(rng.integers(1, 17))
+    p1 = int(rng.integers(1, 12))
+    R1 = int(rng.integers(1, max(2, 2 * WX // p1)))
+    nw1, len1, st1, d1 = windows(L1)
+    o1 = [0] * (n - 2) + [int(rng.integers(-2 * HX, 2 * HX + 1)), int(rng.integers(-2 * WX, 2 * WX + 1))]
+    if seed % 3 == 0:
+        o1[-1] = 4 * int(rng.integers(-WX // 2, WX // 2 + 1))
+    WY = nw1 * R1
+    L2 = int(rng.integers(1, 17))
+    p2 = int(rng.integers(1, L2 + 1))
+    R2 = int(rng.integers(1, 12))
+    nw2, len2, st2, d2 = windows(L2)
+    o2 = [0] * (n - 2) + [int(rng.integers(-2 * HX, 2 * HX + 1)), 0]
+    ones = [1] * (n - 2)
+    e_col = [[0]] * (n - 1) + [[1]]
+    e_row = [[0]] * (n - 2) + [[1], [0]]
+    ax, ay, az = lead + [HX, WX], lead + [HX, WY], lead + [nw2 * R2, WY]
+    t1i = (ax, lead + [HX, R1], [L1], o1, _eye(n, ones + [1, p1]), e_col)
+    t1o = (ay, lead + [HX, R1], [nw1], [0] * n, _eye(n, ones + [1, nw1]), e_col)
+    t2i = (ay, lead + [R2, WY], [L2], o2, _eye(n, ones + [p2, 1]), e_row)
+    t2o = (az, lead + [R2, WY], [nw2], [0] * n, _eye(n, ones + [nw2, 1]), e_row)
+    xh = np.asarray(rng.integers(-3000, 3000, size=ax)).astype(np.int32)
+    y = orc.scatter(orc.make_tiler(*t1o), _task_c(orc.gather(orc.make_tiler(*t1i), xh), st1, len1, d1),
+                    np.zeros(ay, np.int32))
+    bg = np.full(az, -7, np.int32)
+    want = orc.scatter(orc.make_tiler(*t2o), _task_c(orc.gather(orc.make_tiler(*t2i), y), st2, len2, d2), bg)
+    f1 = aol.make_filter(aol.make_tiler(*t1i), aol.make_tiler(*t1o), st1, len1, d1)
+    f2 = aol.make_filter(aol.make_tiler(*t2i), aol.make_tiler(*t2o), st2, len2, d2)
+    out = torch.from_numpy(bg.copy()).cuda()
+    aol.filter_chain_apply(f1, f2, torch.from_numpy(xh).cuda(), out=out)
+    torch.cuda.synchronize()
+    assert aol.last_kernel() == "sep_chain_kernel"
     assert np.array_equal(out.cpu().numpy(), want)
 
 

@@ -45,10 +45,12 @@ peak = float(json.load(open(os.path.join(os.path.dirname(os.path.dirname(os.path
 b = N * C * (H * W + 480 * 720) * 4
 t2 = timed(lambda: (aol.filter_apply(fh, x, out=y), aol.filter_apply(fv, y, out=z)))
 tc = timed(lambda: aol.filter_chain_apply(fh, fv, x, out=z2))
+chain_kernel = aol.last_kernel()
 zf, _ = aol.downscale_frame(x.reshape(N, C, H, W))
 tf = timed(lambda: aol.downscale_frame(x.reshape(N, C, H, W), out=zf))
 same = bool(torch.equal(z, z2) and torch.equal(z2, zf.reshape(P, 480, 720)))
-for name, t in (("f3 generic filters, two launches (Y through HBM)", t2), ("f3 fused chain (one launch)", tc),
+for name, t in (("f3 generic filters, two launches (Y through HBM)", t2),
+                (f"f3 fused chain (one launch, {chain_kernel})", tc),
                 ("d2 specialised fused kernel", tf)):
     print(json.dumps({"config": name, "frames": N, "ms": t, "frames_per_s": N / t * 1e3, "GBps": b / t / 1e6,
                       "frac": b / t / 1e6 / peak, "equal": same}), flush=True)
