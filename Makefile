@@ -9,7 +9,7 @@ OBJS      := $(patsubst $(PKG)/csrc/%.cu,$(BUILD)/%.o,$(CSRC))
 LIB       ?= $(PKG)/libaol.so
 ARCH      := -gencode arch=compute_100a,code=sm_100a
 NVFLAGS   := $(ARCH) -O3 -lineinfo -std=c++17 -Xcompiler -fPIC,-fvisibility=hidden -Xptxas -v \
-             --expt-relaxed-constexpr $(EXTRA)
+             --expt-relaxed-constexpr -I $(BUILD) $(EXTRA)
 ORACLE    := oracle/liboracle.so
 SYNTH     := synth/libsynth.so
 
@@ -20,6 +20,13 @@ all: $(LIB) $(ORACLE) $(SYNTH) $(EXAMPLE)
 $(BUILD)/%.o: $(PKG)/csrc/%.cu $(CHDR)
 	@mkdir -p $(BUILD)
 	$(NVCC) $(NVFLAGS) -c -o $@ $< 2> $(BUILD)/$*.ptxas.log || (cat $(BUILD)/$*.ptxas.log; exit 1)
+
+# the separable chain kernel's body as a string literal, compiled again at run time by NVRTC (chain_sep.cu)
+$(BUILD)/sep_body.inc: $(PKG)/csrc/sep_body.cuh
+	@mkdir -p $(BUILD)
+	{ printf 'R"AOLSEPBODY('; cat $<; printf ')AOLSEPBODY"\n'; } > $@
+
+$(BUILD)/chain_sep.o: $(BUILD)/sep_body.inc
 
 $(LIB): $(OBJS)
 	$(NVCC) $(ARCH) -shared -cudart static -o $@.tmp $(OBJS) -lrt -ldl -lpthread

@@ -39,6 +39,10 @@ AOL_API void aol_debug_fail_next_launches(int n);
  * descriptor or shape takes. */
 AOL_API const char* aol_debug_last_kernel(void);
 
+/* Test hook: aol_filter_chain_apply's separable chains run the kernel specialised at run time by NVRTC (on,
+ * the default unless AOL_CHAIN_JIT=0) or the statically compiled generic one (off).  Same results. */
+AOL_API void aol_debug_set_chain_jit(int on);
+
 #ifdef __cplusplus
 }
 #endif

@@ -22,11 +22,18 @@
 // kernel's constant bank (one IMAD per pattern element and window, no dynamic register indexing); the task is
 // C's S/d - S%d with d by a magic number.
 #include <cuda_runtime.h>
+#include <dlfcn.h>
 
 #include <algorithm>
+#include <atomic>
 #include <cstdint>
+#include <cstdio>
 #include <cstdlib>
 #include <cstring>
+#include <mutex>
+#include <string>
+#include <unordered_map>
+#include <vector>
 
 #include "common.h"
 #include "ptx.cuh"
@@ -34,159 +41,14 @@
 namespace aol {
 namespace {
 
-constexpr int kSepNP = 16;    // pattern elements (L1, L2 <= 16)
-constexpr int kSepNW = 8;     // windows per repetition
-constexpr int kSepNB = 4;     // X row buffers (kSepNB - 1 rows in flight per CTA)
-constexpr int kSepThreads = 256;
-
-struct SepDev {
-    int32_t HX, WX, HY, WY, HZ;
-    int32_t p1, L1, nw1, o1r, o1c, R1;
-    int32_t p2, L2, nw2, o2r, R2;
-    int32_t d1, d2;
-    uint32_t d1_mul, d1_sh, d2_mul, d2_sh;
-    int32_t nb, runs, nunits;
-    int32_t J, xstride, vec;   // staged row length, buffer stride (elements), 16-byte staging
-    int32_t m1[kSepNW][kSepNP], m2[kSepNW][kSepNP];   // window masks
-};
-
-__device__ __forceinline__ int32_t sep_task(int32_t S, int32_t d, uint32_t mul, uint32_t sh) {
-    // C: S/d - S%d = q (1 + d) - S with q = S/d truncated; |S| / |d| by a magic number
-    const uint32_t a = uint32_t(S < 0 ? -S : S);
-    const uint32_t qa = (__umulhi(a, mul) + a) >> sh;
-    const int32_t q = ((S < 0) != (d < 0)) ? -int32_t(qa) : int32_t(qa);
-    return q * (1 + d) - S;
-}
-
-// Window k's sum of a pattern held in registers: a dot product with the k-th 0/1 mask (constant bank).
-template <int NP, int K>
-__device__ __forceinline__ int32_t sep_dot(const int32_t (&x)[NP], const int32_t (&m)[kSepNW][kSepNP]) {
-    int32_t S = 0;
-#pragma unroll
-    for (int p = 0; p < NP; ++p) S += x[p] * m[K][p];
-    return S;
-}
-
-// out(k, task(window k)) for the first nw windows: a jump into a fall-through chain (nw is uniform), so only
-// nw windows' multiply-adds issue (an unrolled loop guarded by k < nw was if-converted: all 8 issued).
-template <int NP, typename Out>
-__device__ __forceinline__ void sep_windows(const int32_t (&x)[NP], const int32_t (&m)[kSepNW][kSepNP], int nw,
-                                            int32_t d, uint32_t mul, uint32_t sh, Out out) {
-    switch (nw) {
-        default:
-        case 8: out(7, sep_task(sep_dot<NP, 7>(x, m), d, mul, sh)); [[fallthrough]];
-        case 7: out(6, sep_task(sep_dot<NP, 6>(x, m), d, mul, sh)); [[fallthrough]];
-        case 6: out(5, sep_task(sep_dot<NP, 5>(x, m), d, mul, sh)); [[fallthrough]];
-        case 5: out(4, sep_task(sep_dot<NP, 4>(x, m), d, mul, sh)); [[fallthrough]];
-        case 4: out(3, sep_task(sep_dot<NP, 3>(x, m), d, mul, sh)); [[fallthrough]];
-        case 3: out(2, sep_task(sep_dot<NP, 2>(x, m), d, mul, sh)); [[fallthrough]];
-        case 2: out(1, sep_task(sep_dot<NP, 1>(x, m), d, mul, sh)); [[fallthrough]];
-        case 1: out(0, sep_task(sep_dot<NP, 0>(x, m), d, mul, sh));
-    }
-}
+#include "sep_body.cuh"
 
 template <int NP1, int NP2>
 __global__ void __launch_bounds__(kSepThreads) sep_chain_kernel(const __grid_constant__ SepDev sd,
                                                                 const int32_t* __restrict__ X,
                                                                 int32_t* __restrict__ Z) {
     extern __shared__ __align__(16) int32_t sm[];
-    int32_t* ring = sm;                                             // [L2][WY]
-    int32_t* xb = sm + ((sd.L2 * sd.WY + 3) & ~3);                  // [kSepNB][xstride]
-    const int tid = threadIdx.x;
-    for (int32_t unit = blockIdx.x; unit < sd.nunits; unit += gridDim.x) {
-        const int32_t plane = unit / sd.runs, run = unit - plane * sd.runs;
-        const int32_t b0 = run * sd.nb, b1 = min(b0 + sd.nb, sd.R2);
-        const int32_t nrows = (b1 - b0 - 1) * sd.p2 + sd.L2;
-        const int32_t* Xp = X + int64_t(plane) * sd.HX * sd.WX;
-        int32_t* Zp = Z + int64_t(plane) * sd.HZ * sd.WY;
-        // X row of the next row to stage: Y row (o2r + p2 b0 + j) mod HY comes from X row (that + o1r) mod HX
-        int32_t xrow_next = int32_t((int64_t(sd.o2r) + int64_t(sd.p2) * b0) % sd.HY) + sd.o1r;
-        if (xrow_next >= sd.HX) xrow_next -= sd.HX;
-        int32_t staged = 0;
-
-        auto issue = [&]() {
-            if (staged < nrows) {
-                const int32_t* src = Xp + int64_t(xrow_next) * sd.WX;
-                const uint32_t dst = ptx::smem_u32(xb + (staged % kSepNB) * sd.xstride);
-                if (sd.vec) {   // o1c, WX multiples of 4: every 16-byte chunk lies on one side of the wrap
-                    for (int32_t c = tid; 4 * c < sd.J; c += kSepThreads) {
-                        int32_t col = sd.o1c + 4 * c;
-                        while (col >= sd.WX) col -= sd.WX;
-                        ptx::cp_async<16>(dst + 16u * uint32_t(c), src + col);
-                    }
-                } else {
-                    for (int32_t e = tid; e < sd.J; e += kSepThreads) {
-                        int32_t col = sd.o1c + e;
-                        while (col >= sd.WX) col -= sd.WX;
-                        ptx::cp_async<4>(dst + 4u * uint32_t(e), src + col);
-                    }
-                }
-                ++staged;
-                if (++xrow_next == sd.HX) xrow_next = 0;   // Y rows (and so X rows) advance by one, toroidally
-            }
-            ptx::cp_async_commit();   // (empty groups keep the count uniform)
-        };
-#pragma unroll
-        for (int i = 0; i < kSepNB - 1; ++i) issue();
-        int32_t yslot = 0;        // ring slot of row j (= j mod L2)
-        int32_t phase = -(sd.L2 - 1);   // j - (L2 - 1) mod p2 once >= 0: 0 when row j completes a band
-        int32_t band = b0;
-        for (int32_t j = 0; j < nrows; ++j) {
-            issue();
-            ptx::cp_async_wait<kSepNB - 1>();
-            __syncthreads();   // row j staged by every thread; the previous band's ring reads are done
-            // ---- f1: one Y row from the staged X row
-            {
-                const int32_t* xr = xb + (j % kSepNB) * sd.xstride;
-                int32_t* yr = ring + yslot * sd.WY;
-                for (int32_t q = tid; q < sd.R1; q += kSepThreads) {
-                    int32_t x[NP1];
-                    const int32_t* xp = xr + sd.p1 * q;
-                    if (sd.p1 % 4 == 0) {   // 16-byte aligned pattern: NP1/4 LDS.128 (scalar loads at a stride of
-                                            // p1 words conflict p1/gcd-way on the banks)
-#pragma unroll
-                        for (int v = 0; v < NP1 / 4; ++v) {
-                            const int4 w = reinterpret_cast<const int4*>(xp)[v];
-                            x[4 * v] = w.x;
-                            x[4 * v + 1] = w.y;
-                            x[4 * v + 2] = w.z;
-                            x[4 * v + 3] = w.w;
-                        }
-                    } else {
-#pragma unroll
-                        for (int p = 0; p < NP1; ++p) x[p] = xp[p];
-                    }
-                    int32_t* yq = yr + sd.nw1 * q;
-                    sep_windows<NP1>(x, sd.m1, sd.nw1, sd.d1, sd.d1_mul, sd.d1_sh,
-                                     [&](int k, int32_t v) { yq[k] = v; });
-                }
-            }
-            __syncthreads();   // the Y row is complete
-            // ---- f2: the band whose last pattern row this was
-            if (phase == 0) {
-                int32_t roff[NP2];
-                int32_t slot = yslot + 1 == sd.L2 ? 0 : yslot + 1;   // oldest row of the ring = the band's row 0
-#pragma unroll
-                for (int i = 0; i < NP2; ++i) {
-                    roff[i] = slot * sd.WY;
-                    if (++slot == sd.L2) slot = 0;
-                }
-                int32_t* zb = Zp + int64_t(sd.nw2) * band * sd.WY;
-                for (int32_t x = tid; x < sd.WY; x += kSepThreads) {
-                    int32_t y[NP2];
-#pragma unroll
-                    for (int i = 0; i < NP2; ++i) y[i] = i < sd.L2 ? ring[roff[i] + x] : 0;
-                    sep_windows<NP2>(y, sd.m2, sd.nw2, sd.d2, sd.d2_mul, sd.d2_sh,
-                                     [&](int k, int32_t v) { zb[int64_t(k) * sd.WY + x] = v; });
-                }
-                ++band;
-            }
-            if (++yslot == sd.L2) yslot = 0;
-            if (++phase == sd.p2) phase = 0;
-        }
-        ptx::cp_async_wait<0>();
-        __syncthreads();   // the next unit restages the buffers and the ring
-    }
+    sep_chain_body<NP1, NP2>(sd, X, Z, sm);
 }
 
 using SepFn = void (*)(const SepDev, const int32_t*, int32_t*);
@@ -323,6 +185,131 @@ bool plan_sep(const aol_filter_t* f1, const aol_filter_t* f2, const DeviceInfo& 
     return true;
 }
 
+// ------------------------------------------------------------ run-time specialisation (NVRTC)
+// The kernel body's text (sep_body.cuh, embedded by the build as a raw string literal).
+const char kSepBodySrc[] =
+#include "sep_body.inc"
+    ;
+
+// NVRTC entry points, resolved once with dlopen: libaol.so does not link NVRTC, and runs the static kernel when
+// it is absent or a compilation fails.
+struct Nvrtc {
+    using Create = int (*)(void**, const char*, const char*, int, const char* const*, const char* const*);
+    using Compile = int (*)(void*, int, const char* const*);
+    using Size = int (*)(void*, size_t*);
+    using Get = int (*)(void*, char*);
+    using Destroy = int (*)(void**);
+    Create create = nullptr;
+    Compile compile = nullptr;
+    Size cubin_size = nullptr, log_size = nullptr;
+    Get cubin = nullptr, log = nullptr;
+    Destroy destroy = nullptr;
+    bool ok = false;
+};
+
+const Nvrtc& nvrtc() {
+    static const Nvrtc n = [] {
+        Nvrtc r;
+        void* h = dlopen("libnvrtc.so.12", RTLD_NOW | RTLD_LOCAL);
+        if (!h) h = dlopen("libnvrtc.so", RTLD_NOW | RTLD_LOCAL);
+        if (!h) return r;
+        r.create = reinterpret_cast<Nvrtc::Create>(dlsym(h, "nvrtcCreateProgram"));
+        r.compile = reinterpret_cast<Nvrtc::Compile>(dlsym(h, "nvrtcCompileProgram"));
+        r.cubin_size = reinterpret_cast<Nvrtc::Size>(dlsym(h, "nvrtcGetCUBINSize"));
+        r.cubin = reinterpret_cast<Nvrtc::Get>(dlsym(h, "nvrtcGetCUBIN"));
+        r.log_size = reinterpret_cast<Nvrtc::Size>(dlsym(h, "nvrtcGetProgramLogSize"));
+        r.log = reinterpret_cast<Nvrtc::Get>(dlsym(h, "nvrtcGetProgramLog"));
+        r.destroy = reinterpret_cast<Nvrtc::Destroy>(dlsym(h, "nvrtcDestroyProgram"));
+        r.ok = r.create && r.compile && r.cubin_size && r.cubin && r.log_size && r.log && r.destroy;
+        return r;
+    }();
+    return n;
+}
+
+// The literal parameters the specialised kernel is compiled for (also its cache key).
+std::string sep_preamble(const aol_filter_t* f1, const aol_filter_t* f2, const SepDev& sd) {
+    const int np1 = sd.p1 % 4 == 0 ? (sd.L1 + 3) / 4 * 4 : sd.L1;   // 16-byte pattern loads need NP1 % 4 == 0
+    std::string s = "#define SEP_JIT 1\n";
+    char b[256];
+    std::snprintf(b, sizeof b,
+                  "#define SEP_NP1 %d\n#define SEP_NP2 %d\n#define SEP_P1 %d\n#define SEP_L1 %d\n#define SEP_NW1 %d\n"
+                  "#define SEP_P2 %d\n#define SEP_L2 %d\n#define SEP_NW2 %d\n#define SEP_D1 (%d)\n#define SEP_D2 (%d)\n",
+                  np1, sd.L2, sd.p1, sd.L1, sd.nw1, sd.p2, sd.L2, sd.nw2, sd.d1, sd.d2);
+    s += b;
+    for (int f = 0; f < 2; ++f) {
+        const aol_filter_t* fl = f == 0 ? f1 : f2;
+        const int L = f == 0 ? sd.L1 : sd.L2;
+        std::string starts;
+        for (int k = 0; k < fl->n_windows; ++k) {
+            std::snprintf(b, sizeof b, "k == %d ? %d : ", k, fl->window_start[k]);
+            starts += b;
+        }
+        s += "struct sep_m" + std::to_string(f + 1) +
+             " { __device__ constexpr int operator()(int k, int p) const { return p >= (" + starts + "0) && p < (" +
+             starts + "0) + " + std::to_string(fl->window_len) + " && p < " + std::to_string(L) + "; } };\n";
+    }
+    return s;
+}
+
+std::atomic<int> g_sep_jit{-1};   // -1: from AOL_CHAIN_JIT (default on); 0 / 1: set by aol_debug_set_chain_jit
+
+bool sep_jit_enabled() {
+    int v = g_sep_jit.load();
+    if (v < 0) {
+        const char* e = std::getenv("AOL_CHAIN_JIT");
+        v = (e && e[0] == '0') ? 0 : 1;
+    }
+    return v != 0;
+}
+
+// The specialised kernel for these filters: compiled on first use, then cached (per process; a library loaded
+// through the runtime is available on every device).  nullptr: NVRTC missing or the compilation failed (the
+// reason is kept for aol_last_error-free diagnostics in jit_note).
+std::mutex g_jit_mu;
+std::unordered_map<std::string, const void*> g_jit_cache;
+std::string g_jit_note;
+
+const void* sep_jit_kernel(const aol_filter_t* f1, const aol_filter_t* f2, const SepDev& sd) {
+    if (!sep_jit_enabled()) return nullptr;
+    const Nvrtc& nv = nvrtc();
+    if (!nv.ok) return nullptr;
+    const std::string pre = sep_preamble(f1, f2, sd);
+    std::lock_guard<std::mutex> lock(g_jit_mu);
+    auto it = g_jit_cache.find(pre);
+    if (it != g_jit_cache.end()) return it->second;
+    const void* kern = nullptr;
+    const std::string src = pre + kSepBodySrc;
+    void* prog = nullptr;
+    if (nv.create(&prog, src.c_str(), "aol_sep_chain.cu", 0, nullptr, nullptr) == 0) {
+        const char* opts[] = {"--gpu-architecture=sm_100a", "-std=c++17", "-lineinfo"};
+        if (nv.compile(prog, 3, opts) == 0) {
+            size_t n = 0;
+            nv.cubin_size(prog, &n);
+            std::vector<char> cubin(n);
+            nv.cubin(prog, cubin.data());
+            cudaLibrary_t lib = nullptr;
+            cudaKernel_t k = nullptr;
+            cudaError_t le = cudaLibraryLoadData(&lib, cubin.data(), nullptr, nullptr, 0, nullptr, nullptr, 0);
+            if (le == cudaSuccess) le = cudaLibraryGetKernel(&k, lib, "sep_chain_jit");
+            if (le == cudaSuccess)
+                kern = reinterpret_cast<const void*>(k);   // the library stays loaded for the process
+            else
+                g_jit_note = std::string("loading the compiled kernel failed: ") + cudaGetErrorString(le);
+            cudaGetLastError();
+        } else {
+            size_t n = 0;
+            nv.log_size(prog, &n);
+            std::string log(n, '\0');
+            nv.log(prog, &log[0]);
+            g_jit_note = "NVRTC: " + log;
+        }
+        nv.destroy(&prog);
+    }
+    if (!kern && std::getenv("AOL_JIT_VERBOSE")) std::fprintf(stderr, "aol: chain JIT failed: %s\n", g_jit_note.c_str());
+    g_jit_cache.emplace(pre, kern);   // failures are cached too: the static kernel serves those filters
+    return kern;
+}
+
 }  // namespace
 
 // AOL_CHAIN_SEP=0 disables the separable chain kernel (A/B measurements only).
@@ -343,21 +330,29 @@ bool launch_sep_chain(const aol_filter_t* f1, const aol_filter_t* f2, const int3
     if (sd.vec && reinterpret_cast<uintptr_t>(d_in) % 16) sd.vec = 0;
     *st = AOL_OK;
     if (sd.nunits == 0) return true;
-    const SepFn kern = sep_kernel_for(sd.L1, sd.L2);
-    *st = kernel_smem(reinterpret_cast<const void*>(kern), smem);
+    // the run-time specialised kernel when NVRTC is there, else the static one (same body, parameters read
+    // from the descriptor)
+    const void* jit = sep_jit_kernel(f1, f2, sd);
+    const void* kern = jit ? jit : reinterpret_cast<const void*>(sep_kernel_for(sd.L1, sd.L2));
+    const char* name = jit ? "sep_chain_jit" : "sep_chain_kernel";
+    *st = kernel_smem(kern, smem);
     if (*st != AOL_OK) return true;
-    const int per_sm = std::max(1, kernel_occupancy(reinterpret_cast<const void*>(kern), kSepThreads, smem));
+    const int per_sm = std::max(1, kernel_occupancy(kern, kSepThreads, smem));
     const int grid = int(std::max<int64_t>(1, std::min<int64_t>(sd.nunits, int64_t(dev.num_sms) * per_sm)));
-    *st = launch_preflight(reinterpret_cast<const void*>(kern), kSepThreads, smem, "sep_chain_kernel");
+    *st = launch_preflight(kern, kSepThreads, smem, name);
     if (*st != AOL_OK) return true;
-    kern<<<grid, kSepThreads, smem, s>>>(sd, d_in, d_out);
-    note_launch("sep_chain_kernel");
-    const cudaError_t e = cudaGetLastError();
+    void* args[] = {&sd, const_cast<int32_t**>(&d_in), &d_out};
+    const cudaError_t e = cudaLaunchKernel(kern, dim3(unsigned(grid)), dim3(kSepThreads), args, size_t(smem), s);
+    note_launch(name);
     if (e != cudaSuccess) {
-        set_error("launch of sep_chain_kernel failed: %s", cudaGetErrorString(e));
+        set_error("launch of %s failed: %s", name, cudaGetErrorString(e));
         *st = AOL_E_CUDA;
     }
     return true;
 }
 
+void set_sep_jit(int on) { g_sep_jit.store(on ? 1 : 0); }
+
 }  // namespace aol
+
+extern "C" AOL_API void aol_debug_set_chain_jit(int on) { aol::set_sep_jit(on); }

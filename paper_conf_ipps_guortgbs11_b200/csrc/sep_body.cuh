@@ -1,0 +1,215 @@
+// sep_body.cuh -- the separable chain kernel (chain_sep.cu explains the class and the design), written once and
+// compiled twice:
+//   * statically into libaol.so (SEP_JIT undefined): every filter parameter is read from the SepDev argument --
+//     window sums as dot products with 0/1 masks, the task's division by a magic number;
+//   * per filter pair by NVRTC at run time (SEP_JIT defined, chain_sep.cu prepends the parameters as literal
+//     constants): the masks fold away into plain sums of the window elements, the divisions by constant divisors
+//     into multiply-shifts, the window dispatch and pattern lengths into straight-line code -- what the paper's
+//     SaC compiler does for tilers known at compile time, done for descriptors known only at run time.
+// Self-contained: no headers (NVRTC compiles it without the CUDA toolkit's include tree).
+#ifndef AOL_SEP_BODY
+#define AOL_SEP_BODY
+
+constexpr int kSepNP = 16;    // pattern elements (L1, L2 <= 16)
+constexpr int kSepNW = 8;     // windows per repetition
+constexpr int kSepNB = 4;     // X row buffers (kSepNB - 1 rows in flight per CTA)
+constexpr int kSepThreads = 256;
+
+typedef int sep_i32;
+typedef unsigned int sep_u32;
+typedef long long sep_i64;
+
+struct SepDev {
+    sep_i32 HX, WX, HY, WY, HZ;
+    sep_i32 p1, L1, nw1, o1r, o1c, R1;
+    sep_i32 p2, L2, nw2, o2r, R2;
+    sep_i32 d1, d2;
+    sep_u32 d1_mul, d1_sh, d2_mul, d2_sh;
+    sep_i32 nb, runs, nunits;
+    sep_i32 J, xstride, vec;   // staged row length, buffer stride (elements), 16-byte staging
+    sep_i32 m1[kSepNW][kSepNP], m2[kSepNW][kSepNP];   // window masks (0/1)
+};
+
+#ifdef SEP_JIT
+// NVRTC: SEP_NP1 .. SEP_D2 (literals) and the mask functors sep_m1 / sep_m2 (constexpr, from the literal window
+// starts) are defined ahead of this text
+#define SEP_M1 sep_m1{}
+#define SEP_M2 sep_m2{}
+#define SEP_TASK(S, d, mul, sh) ((S) / (d) - (S) % (d))
+#else
+#define SEP_P1 sd.p1
+#define SEP_L1 sd.L1
+#define SEP_NW1 sd.nw1
+#define SEP_P2 sd.p2
+#define SEP_L2 sd.L2
+#define SEP_NW2 sd.nw2
+#define SEP_D1 sd.d1
+#define SEP_D2 sd.d2
+#define SEP_M1 [&](int k, int p) { return sd.m1[k][p]; }
+#define SEP_M2 [&](int k, int p) { return sd.m2[k][p]; }
+#define SEP_TASK(S, d, mul, sh) sep_task(S, d, mul, sh)
+#endif
+
+// C's S/d - S%d (truncating) = q (1 + d) - S, |S| / |d| by a magic number.
+__device__ __forceinline__ sep_i32 sep_task(sep_i32 S, sep_i32 d, sep_u32 mul, sep_u32 sh) {
+    const sep_u32 a = sep_u32(S < 0 ? -S : S);
+    const sep_u32 qa = (__umulhi(a, mul) + a) >> sh;
+    const sep_i32 q = ((S < 0) != (d < 0)) ? -sep_i32(qa) : sep_i32(qa);
+    return q * (1 + d) - S;
+}
+
+// Window K's sum of a pattern held in registers: a dot product with the K-th 0/1 mask m(K, p).
+template <int NP, int K, typename M>
+__device__ __forceinline__ sep_i32 sep_dot(const sep_i32 (&x)[NP], const M& m) {
+    sep_i32 S = 0;
+#pragma unroll
+    for (int p = 0; p < NP; ++p) S += x[p] * m(K, p);
+    return S;
+}
+
+// out(k, window k's task value) for the first nw windows: a jump into a fall-through chain (nw is uniform), so
+// only nw windows' multiply-adds issue (an unrolled loop guarded by k < nw was if-converted: all 8 issued).
+#define SEP_W(K, NP, x, m, d, mul, sh, out) out(K, SEP_TASK((sep_dot<NP, K>(x, m)), d, mul, sh))
+template <int NP, typename M, typename Out>
+__device__ __forceinline__ void sep_windows(const sep_i32 (&x)[NP], M m, int nw, sep_i32 d, sep_u32 mul,
+                                            sep_u32 sh, Out out) {
+    switch (nw) {
+        default:
+        case 8: SEP_W(7, NP, x, m, d, mul, sh, out); [[fallthrough]];
+        case 7: SEP_W(6, NP, x, m, d, mul, sh, out); [[fallthrough]];
+        case 6: SEP_W(5, NP, x, m, d, mul, sh, out); [[fallthrough]];
+        case 5: SEP_W(4, NP, x, m, d, mul, sh, out); [[fallthrough]];
+        case 4: SEP_W(3, NP, x, m, d, mul, sh, out); [[fallthrough]];
+        case 3: SEP_W(2, NP, x, m, d, mul, sh, out); [[fallthrough]];
+        case 2: SEP_W(1, NP, x, m, d, mul, sh, out); [[fallthrough]];
+        case 1: SEP_W(0, NP, x, m, d, mul, sh, out);
+    }
+}
+#undef SEP_W
+
+__device__ __forceinline__ void sep_cp_async16(sep_u32 saddr, const void* g) {
+    asm volatile("cp.async.cg.shared.global [%0], [%1], 16;" ::"r"(saddr), "l"(g) : "memory");
+}
+__device__ __forceinline__ void sep_cp_async4(sep_u32 saddr, const void* g) {
+    asm volatile("cp.async.ca.shared.global [%0], [%1], 4;" ::"r"(saddr), "l"(g) : "memory");
+}
+__device__ __forceinline__ void sep_cp_commit() { asm volatile("cp.async.commit_group;" ::: "memory"); }
+template <int N>
+__device__ __forceinline__ void sep_cp_wait() { asm volatile("cp.async.wait_group %0;" ::"n"(N) : "memory"); }
+__device__ __forceinline__ sep_u32 sep_smem_u32(const void* p) {
+    return sep_u32(__cvta_generic_to_shared(p));
+}
+
+template <int NP1, int NP2>
+__device__ __forceinline__ void sep_chain_body(const SepDev& sd, const sep_i32* __restrict__ X,
+                                               sep_i32* __restrict__ Z, sep_i32* sm) {
+    sep_i32* ring = sm;                                             // [L2][WY]
+    sep_i32* xb = sm + ((SEP_L2 * sd.WY + 3) & ~3);                 // [kSepNB][xstride]
+    const int tid = threadIdx.x;
+    for (sep_i32 unit = blockIdx.x; unit < sd.nunits; unit += gridDim.x) {
+        const sep_i32 plane = unit / sd.runs, run = unit - plane * sd.runs;
+        const sep_i32 b0 = run * sd.nb, b1 = min(b0 + sd.nb, sd.R2);
+        const sep_i32 nrows = (b1 - b0 - 1) * SEP_P2 + SEP_L2;
+        const sep_i32* Xp = X + sep_i64(plane) * sd.HX * sd.WX;
+        sep_i32* Zp = Z + sep_i64(plane) * sd.HZ * sd.WY;
+        // X row of the next row to stage: Y row (o2r + p2 b0 + j) mod HY comes from X row (that + o1r) mod HX
+        sep_i32 xrow_next = sep_i32((sep_i64(sd.o2r) + sep_i64(SEP_P2) * b0) % sd.HY) + sd.o1r;
+        if (xrow_next >= sd.HX) xrow_next -= sd.HX;
+        sep_i32 staged = 0;
+
+        auto issue = [&]() {
+            if (staged < nrows) {
+                const sep_i32* src = Xp + sep_i64(xrow_next) * sd.WX;
+                const sep_u32 dst = sep_smem_u32(xb + (staged % kSepNB) * sd.xstride);
+                if (sd.vec) {   // o1c, WX multiples of 4: every 16-byte chunk lies on one side of the wrap
+                    for (sep_i32 c = tid; 4 * c < sd.J; c += kSepThreads) {
+                        sep_i32 col = sd.o1c + 4 * c;
+                        while (col >= sd.WX) col -= sd.WX;
+                        sep_cp_async16(dst + 16u * sep_u32(c), src + col);
+                    }
+                } else {
+                    for (sep_i32 e = tid; e < sd.J; e += kSepThreads) {
+                        sep_i32 col = sd.o1c + e;
+                        while (col >= sd.WX) col -= sd.WX;
+                        sep_cp_async4(dst + 4u * sep_u32(e), src + col);
+                    }
+                }
+                ++staged;
+                if (++xrow_next == sd.HX) xrow_next = 0;   // Y rows (and so X rows) advance by one, toroidally
+            }
+            sep_cp_commit();   // (empty groups keep the count uniform)
+        };
+#pragma unroll
+        for (int i = 0; i < kSepNB - 1; ++i) issue();
+        sep_i32 yslot = 0;                // ring slot of row j (= j mod L2)
+        sep_i32 phase = -(SEP_L2 - 1);    // (j - (L2 - 1)) mod p2 once >= 0: 0 when row j completes a band
+        sep_i32 band = b0;
+        for (sep_i32 j = 0; j < nrows; ++j) {
+            issue();
+            sep_cp_wait<kSepNB - 1>();
+            __syncthreads();   // row j staged by every thread; the previous band's ring reads are done
+            // ---- f1: one Y row from the staged X row
+            {
+                const sep_i32* xr = xb + (j % kSepNB) * sd.xstride;
+                sep_i32* yr = ring + yslot * sd.WY;
+                for (sep_i32 q = tid; q < sd.R1; q += kSepThreads) {
+                    sep_i32 x[NP1];
+                    const sep_i32* xp = xr + SEP_P1 * q;
+                    if (NP1 % 4 == 0 && SEP_P1 % 4 == 0) {
+                        // 16-byte aligned pattern: NP1/4 LDS.128 (scalar loads at a stride of p1 words conflict
+                        // p1/gcd-way on the banks)
+#pragma unroll
+                        for (int v = 0; v < NP1 / 4; ++v) {
+                            const int4 w = reinterpret_cast<const int4*>(xp)[v];
+                            x[4 * v] = w.x;
+                            x[4 * v + 1] = w.y;
+                            x[4 * v + 2] = w.z;
+                            x[4 * v + 3] = w.w;
+                        }
+                    } else {
+#pragma unroll
+                        for (int p = 0; p < NP1; ++p) x[p] = xp[p];
+                    }
+                    sep_i32* yq = yr + SEP_NW1 * q;
+                    sep_windows<NP1>(x, SEP_M1, SEP_NW1, SEP_D1, sd.d1_mul, sd.d1_sh,
+                                     [&](int k, sep_i32 v) { yq[k] = v; });
+                }
+            }
+            __syncthreads();   // the Y row is complete
+            // ---- f2: the band whose last pattern row this was
+            if (phase == 0) {
+                sep_i32 roff[NP2];
+                sep_i32 slot = yslot + 1 == SEP_L2 ? 0 : yslot + 1;   // oldest row of the ring = the band's row 0
+#pragma unroll
+                for (int i = 0; i < NP2; ++i) {
+                    roff[i] = slot * sd.WY;
+                    if (++slot == SEP_L2) slot = 0;
+                }
+                sep_i32* zb = Zp + sep_i64(SEP_NW2) * band * sd.WY;
+                for (sep_i32 x = tid; x < sd.WY; x += kSepThreads) {
+                    sep_i32 y[NP2];
+#pragma unroll
+                    for (int i = 0; i < NP2; ++i) y[i] = i < SEP_L2 ? ring[roff[i] + x] : 0;
+                    sep_windows<NP2>(y, SEP_M2, SEP_NW2, SEP_D2, sd.d2_mul, sd.d2_sh,
+                                     [&](int k, sep_i32 v) { zb[sep_i64(k) * sd.WY + x] = v; });
+                }
+                ++band;
+            }
+            if (++yslot == SEP_L2) yslot = 0;
+            if (++phase == SEP_P2) phase = 0;
+        }
+        sep_cp_wait<0>();
+        __syncthreads();   // the next unit restages the buffers and the ring
+    }
+}
+
+#ifdef SEP_JIT
+extern "C" __global__ void __launch_bounds__(kSepThreads) sep_chain_jit(const __grid_constant__ SepDev sd,
+                                                                        const sep_i32* __restrict__ X,
+                                                                        sep_i32* __restrict__ Z) {
+    extern __shared__ __align__(16) sep_i32 sep_sm[];
+    sep_chain_body<SEP_NP1, SEP_NP2>(sd, X, Z, sep_sm);
+}
+#endif
+
+#endif  // AOL_SEP_BODY

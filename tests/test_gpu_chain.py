@@ -31,7 +31,7 @@ def test_chain_h_then_v_equals_fused_downscaler(orc, shape):
     fv = aol.filter_preset(aol.FILTER_V, P, H, 3 * W // 8)
     z = aol.filter_chain_apply(fh, fv, x)
     torch.cuda.synchronize()
-    assert aol.last_kernel() == "sep_chain_kernel"
+    assert aol.last_kernel() == "sep_chain_jit"
     zf, _ = aol.downscale_frame(x.unsqueeze(1))
     assert torch.equal(z, zf[:, 0])
     if H * W <= 1080 * 1920:
@@ -111,7 +111,7 @@ def test_random_chains(orc, seed):
     out = torch.from_numpy(bg.copy()).cuda()
     aol.filter_chain_apply(f1, f2, torch.from_numpy(xh).cuda(), out=out)
     torch.cuda.synchronize()
-    assert aol.last_kernel() in ("chain_kernel", "sep_chain_kernel")
+    assert aol.last_kernel() in ("chain_kernel", "sep_chain_kernel", "sep_chain_jit")
     assert np.array_equal(out.cpu().numpy(), want)
 
 
@@ -124,7 +124,8 @@ def test_random_separable_chains(orc, seed):
     """A row filter then a column filter with every parameter random: lead dims (planes), pattern lengths <= 16,
     paving steps (patterns overlapping, abutting or leaving gaps along the row; p2 <= L2 down the columns),
     origins wrapping the row several times and shifting the rows, 1-8 windows, divisors of either sign, column
-    origins on and off the 16-byte grid.  Expected: the oracle's gather -> C task -> scatter, twice."""
+    origins on and off the 16-byte grid.  Expected: the oracle's gather -> C task -> scatter, twice.  Even seeds
+    run the kernel specialised at run time (NVRTC), odd seeds the statically compiled one."""
     rng = np.random.default_rng(7700 + seed)
     n = int(rng.integers(2, 5))
     lead = [int(rng.integers(1, 4)) for _ in range(n - 2)]
@@ -166,9 +167,14 @@ def test_random_separable_chains(orc, seed):
     f1 = aol.make_filter(aol.make_tiler(*t1i), aol.make_tiler(*t1o), st1, len1, d1)
     f2 = aol.make_filter(aol.make_tiler(*t2i), aol.make_tiler(*t2o), st2, len2, d2)
     out = torch.from_numpy(bg.copy()).cuda()
-    aol.filter_chain_apply(f1, f2, torch.from_numpy(xh).cuda(), out=out)
-    torch.cuda.synchronize()
-    assert aol.last_kernel() == "sep_chain_kernel"
+    jit = seed % 2 == 0
+    aol._lib.lib().aol_debug_set_chain_jit(int(jit))
+    try:
+        aol.filter_chain_apply(f1, f2, torch.from_numpy(xh).cuda(), out=out)
+        torch.cuda.synchronize()
+        assert aol.last_kernel() == ("sep_chain_jit" if jit else "sep_chain_kernel")
+    finally:
+        aol._lib.lib().aol_debug_set_chain_jit(1)
     assert np.array_equal(out.cpu().numpy(), want)
 
 
