@@ -226,7 +226,8 @@ const Nvrtc& nvrtc() {
     return n;
 }
 
-// The literal parameters the specialised kernel is compiled for (also its cache key).
+// The literal parameters the specialised kernel is compiled for (also its cache key): the filters' patterns,
+// windows and divisors, and the array shapes (a video's frame size is fixed; a new one compiles once more).
 std::string sep_preamble(const aol_filter_t* f1, const aol_filter_t* f2, const SepDev& sd) {
     const int np1 = sd.p1 % 4 == 0 ? (sd.L1 + 3) / 4 * 4 : sd.L1;   // 16-byte pattern loads need NP1 % 4 == 0
     std::string s = "#define SEP_JIT 1\n";
@@ -235,6 +236,11 @@ std::string sep_preamble(const aol_filter_t* f1, const aol_filter_t* f2, const S
                   "#define SEP_NP1 %d\n#define SEP_NP2 %d\n#define SEP_P1 %d\n#define SEP_L1 %d\n#define SEP_NW1 %d\n"
                   "#define SEP_P2 %d\n#define SEP_L2 %d\n#define SEP_NW2 %d\n#define SEP_D1 (%d)\n#define SEP_D2 (%d)\n",
                   np1, sd.L2, sd.p1, sd.L1, sd.nw1, sd.p2, sd.L2, sd.nw2, sd.d1, sd.d2);
+    s += b;
+    std::snprintf(b, sizeof b,
+                  "#define SEP_HX %d\n#define SEP_WX %d\n#define SEP_HY %d\n#define SEP_WY %d\n#define SEP_HZ %d\n"
+                  "#define SEP_R1 %d\n#define SEP_J %d\n#define SEP_XSTRIDE %d\n#define SEP_VEC %d\n#define SEP_O1C %d\n",
+                  sd.HX, sd.WX, sd.HY, sd.WY, sd.HZ, sd.R1, sd.J, sd.xstride, sd.vec, sd.o1c);
     s += b;
     for (int f = 0; f < 2; ++f) {
         const aol_filter_t* fl = f == 0 ? f1 : f2;

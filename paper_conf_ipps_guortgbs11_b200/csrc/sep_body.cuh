@@ -31,8 +31,8 @@ struct SepDev {
 };
 
 #ifdef SEP_JIT
-// NVRTC: SEP_NP1 .. SEP_D2 (literals) and the mask functors sep_m1 / sep_m2 (constexpr, from the literal window
-// starts) are defined ahead of this text
+// NVRTC: SEP_NP1 .. SEP_D2, the array shapes SEP_HX .. SEP_O1C (literals) and the mask functors sep_m1 / sep_m2
+// (constexpr, from the literal window starts) are defined ahead of this text
 #define SEP_M1 sep_m1{}
 #define SEP_M2 sep_m2{}
 #define SEP_TASK(S, d, mul, sh) ((S) / (d) - (S) % (d))
@@ -45,6 +45,16 @@ struct SepDev {
 #define SEP_NW2 sd.nw2
 #define SEP_D1 sd.d1
 #define SEP_D2 sd.d2
+#define SEP_HX sd.HX
+#define SEP_WX sd.WX
+#define SEP_HY sd.HY
+#define SEP_WY sd.WY
+#define SEP_HZ sd.HZ
+#define SEP_R1 sd.R1
+#define SEP_J sd.J
+#define SEP_XSTRIDE sd.xstride
+#define SEP_VEC sd.vec
+#define SEP_O1C sd.o1c
 #define SEP_M1 [&](int k, int p) { return sd.m1[k][p]; }
 #define SEP_M2 [&](int k, int p) { return sd.m2[k][p]; }
 #define SEP_TASK(S, d, mul, sh) sep_task(S, d, mul, sh)
@@ -104,38 +114,38 @@ template <int NP1, int NP2>
 __device__ __forceinline__ void sep_chain_body(const SepDev& sd, const sep_i32* __restrict__ X,
                                                sep_i32* __restrict__ Z, sep_i32* sm) {
     sep_i32* ring = sm;                                             // [L2][WY]
-    sep_i32* xb = sm + ((SEP_L2 * sd.WY + 3) & ~3);                 // [kSepNB][xstride]
+    sep_i32* xb = sm + ((SEP_L2 * SEP_WY + 3) & ~3);                 // [kSepNB][xstride]
     const int tid = threadIdx.x;
     for (sep_i32 unit = blockIdx.x; unit < sd.nunits; unit += gridDim.x) {
         const sep_i32 plane = unit / sd.runs, run = unit - plane * sd.runs;
         const sep_i32 b0 = run * sd.nb, b1 = min(b0 + sd.nb, sd.R2);
         const sep_i32 nrows = (b1 - b0 - 1) * SEP_P2 + SEP_L2;
-        const sep_i32* Xp = X + sep_i64(plane) * sd.HX * sd.WX;
-        sep_i32* Zp = Z + sep_i64(plane) * sd.HZ * sd.WY;
+        const sep_i32* Xp = X + sep_i64(plane) * SEP_HX * SEP_WX;
+        sep_i32* Zp = Z + sep_i64(plane) * SEP_HZ * SEP_WY;
         // X row of the next row to stage: Y row (o2r + p2 b0 + j) mod HY comes from X row (that + o1r) mod HX
-        sep_i32 xrow_next = sep_i32((sep_i64(sd.o2r) + sep_i64(SEP_P2) * b0) % sd.HY) + sd.o1r;
-        if (xrow_next >= sd.HX) xrow_next -= sd.HX;
+        sep_i32 xrow_next = sep_i32((sep_i64(sd.o2r) + sep_i64(SEP_P2) * b0) % SEP_HY) + sd.o1r;
+        if (xrow_next >= SEP_HX) xrow_next -= SEP_HX;
         sep_i32 staged = 0;
 
         auto issue = [&]() {
             if (staged < nrows) {
-                const sep_i32* src = Xp + sep_i64(xrow_next) * sd.WX;
-                const sep_u32 dst = sep_smem_u32(xb + (staged % kSepNB) * sd.xstride);
-                if (sd.vec) {   // o1c, WX multiples of 4: every 16-byte chunk lies on one side of the wrap
-                    for (sep_i32 c = tid; 4 * c < sd.J; c += kSepThreads) {
-                        sep_i32 col = sd.o1c + 4 * c;
-                        while (col >= sd.WX) col -= sd.WX;
+                const sep_i32* src = Xp + sep_i64(xrow_next) * SEP_WX;
+                const sep_u32 dst = sep_smem_u32(xb + (staged % kSepNB) * SEP_XSTRIDE);
+                if (SEP_VEC) {   // o1c, WX multiples of 4: every 16-byte chunk lies on one side of the wrap
+                    for (sep_i32 c = tid; 4 * c < SEP_J; c += kSepThreads) {
+                        sep_i32 col = SEP_O1C + 4 * c;
+                        while (col >= SEP_WX) col -= SEP_WX;
                         sep_cp_async16(dst + 16u * sep_u32(c), src + col);
                     }
                 } else {
-                    for (sep_i32 e = tid; e < sd.J; e += kSepThreads) {
-                        sep_i32 col = sd.o1c + e;
-                        while (col >= sd.WX) col -= sd.WX;
+                    for (sep_i32 e = tid; e < SEP_J; e += kSepThreads) {
+                        sep_i32 col = SEP_O1C + e;
+                        while (col >= SEP_WX) col -= SEP_WX;
                         sep_cp_async4(dst + 4u * sep_u32(e), src + col);
                     }
                 }
                 ++staged;
-                if (++xrow_next == sd.HX) xrow_next = 0;   // Y rows (and so X rows) advance by one, toroidally
+                if (++xrow_next == SEP_HX) xrow_next = 0;   // Y rows (and so X rows) advance by one, toroidally
             }
             sep_cp_commit();   // (empty groups keep the count uniform)
         };
@@ -150,9 +160,9 @@ __device__ __forceinline__ void sep_chain_body(const SepDev& sd, const sep_i32* 
             __syncthreads();   // row j staged by every thread; the previous band's ring reads are done
             // ---- f1: one Y row from the staged X row
             {
-                const sep_i32* xr = xb + (j % kSepNB) * sd.xstride;
-                sep_i32* yr = ring + yslot * sd.WY;
-                for (sep_i32 q = tid; q < sd.R1; q += kSepThreads) {
+                const sep_i32* xr = xb + (j % kSepNB) * SEP_XSTRIDE;
+                sep_i32* yr = ring + yslot * SEP_WY;
+                for (sep_i32 q = tid; q < SEP_R1; q += kSepThreads) {
                     sep_i32 x[NP1];
                     const sep_i32* xp = xr + SEP_P1 * q;
                     if (NP1 % 4 == 0 && SEP_P1 % 4 == 0) {
@@ -182,16 +192,16 @@ __device__ __forceinline__ void sep_chain_body(const SepDev& sd, const sep_i32* 
                 sep_i32 slot = yslot + 1 == SEP_L2 ? 0 : yslot + 1;   // oldest row of the ring = the band's row 0
 #pragma unroll
                 for (int i = 0; i < NP2; ++i) {
-                    roff[i] = slot * sd.WY;
+                    roff[i] = slot * SEP_WY;
                     if (++slot == SEP_L2) slot = 0;
                 }
-                sep_i32* zb = Zp + sep_i64(SEP_NW2) * band * sd.WY;
-                for (sep_i32 x = tid; x < sd.WY; x += kSepThreads) {
+                sep_i32* zb = Zp + sep_i64(SEP_NW2) * band * SEP_WY;
+                for (sep_i32 x = tid; x < SEP_WY; x += kSepThreads) {
                     sep_i32 y[NP2];
 #pragma unroll
                     for (int i = 0; i < NP2; ++i) y[i] = i < SEP_L2 ? ring[roff[i] + x] : 0;
                     sep_windows<NP2>(y, SEP_M2, SEP_NW2, SEP_D2, sd.d2_mul, sd.d2_sh,
-                                     [&](int k, sep_i32 v) { zb[sep_i64(k) * sd.WY + x] = v; });
+                                     [&](int k, sep_i32 v) { zb[sep_i64(k) * SEP_WY + x] = v; });
                 }
                 ++band;
             }
