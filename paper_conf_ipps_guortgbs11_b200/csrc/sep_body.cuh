@@ -131,16 +131,24 @@ __device__ __forceinline__ void sep_chain_body(const SepDev& sd, const sep_i32* 
             if (staged < nrows) {
                 const sep_i32* src = Xp + sep_i64(xrow_next) * SEP_WX;
                 const sep_u32 dst = sep_smem_u32(xb + (staged % kSepNB) * SEP_XSTRIDE);
+                // (one conditional subtraction when the staged span wraps at most once, o1c + J <= 2 WX)
+                const bool once = SEP_O1C + SEP_J <= 2 * SEP_WX;
                 if (SEP_VEC) {   // o1c, WX multiples of 4: every 16-byte chunk lies on one side of the wrap
                     for (sep_i32 c = tid; 4 * c < SEP_J; c += kSepThreads) {
                         sep_i32 col = SEP_O1C + 4 * c;
-                        while (col >= SEP_WX) col -= SEP_WX;
+                        if (once)
+                            col -= col >= SEP_WX ? SEP_WX : 0;
+                        else
+                            while (col >= SEP_WX) col -= SEP_WX;
                         sep_cp_async16(dst + 16u * sep_u32(c), src + col);
                     }
                 } else {
                     for (sep_i32 e = tid; e < SEP_J; e += kSepThreads) {
                         sep_i32 col = SEP_O1C + e;
-                        while (col >= SEP_WX) col -= SEP_WX;
+                        if (once)
+                            col -= col >= SEP_WX ? SEP_WX : 0;
+                        else
+                            while (col >= SEP_WX) col -= SEP_WX;
                         sep_cp_async4(dst + 4u * sep_u32(e), src + col);
                     }
                 }
@@ -167,14 +175,25 @@ __device__ __forceinline__ void sep_chain_body(const SepDev& sd, const sep_i32* 
                     const sep_i32* xp = xr + SEP_P1 * q;
                     if (NP1 % 4 == 0 && SEP_P1 % 4 == 0) {
                         // 16-byte aligned pattern: NP1/4 LDS.128 (scalar loads at a stride of p1 words conflict
-                        // p1/gcd-way on the banks)
+                        // p1/gcd-way on the banks).  At p1 = 8 a quarter-warp's chunks v sit in every other
+                        // 16-byte bank group: lanes with bit 2 set take chunks 0 and 1 in the other order, which
+                        // spreads both loads over all 8 groups (conflict-free).
+                        const bool swp = SEP_P1 == 8 && ((tid >> 2) & 1);
+                        const int4* xp4 = reinterpret_cast<const int4*>(xp);
+                        int4 c[NP1 / 4 > 0 ? NP1 / 4 : 1];
+#pragma unroll
+                        for (int v = 0; v < NP1 / 4; ++v) c[v] = xp4[v];
+                        if (NP1 >= 8) {
+                            const int4 L0 = xp4[swp ? 1 : 0], L1 = xp4[swp ? 0 : 1];   // load slots 0 and 1
+                            c[0] = swp ? L1 : L0;
+                            c[1] = swp ? L0 : L1;
+                        }
 #pragma unroll
                         for (int v = 0; v < NP1 / 4; ++v) {
-                            const int4 w = reinterpret_cast<const int4*>(xp)[v];
-                            x[4 * v] = w.x;
-                            x[4 * v + 1] = w.y;
-                            x[4 * v + 2] = w.z;
-                            x[4 * v + 3] = w.w;
+                            x[4 * v] = c[v].x;
+                            x[4 * v + 1] = c[v].y;
+                            x[4 * v + 2] = c[v].z;
+                            x[4 * v + 3] = c[v].w;
                         }
                     } else {
 #pragma unroll
