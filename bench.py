@@ -25,7 +25,9 @@ host enqueue), d3 (generic tiler gather / FAST / SEQUENTIAL scatter on the
 SURVEY instance, a wrapping variant and the paper's H input tiler), d4 (64 4K
 frames), d5 (the 10,000-frame stream frame-sharded over the N ranks: strong
 scaling, at every N; every stream frame's checksum verified), wide (16 8K DCI
-frames, 8192 wide: the fused kernel's column strips).
+frames, 8192 wide: the fused kernel's column strips), f3 (the same 300 frames
+through the paper's H and V filters as run-time descriptors, chained into one
+kernel specialised at run time; its checksums must equal the d2 kernel's).
 
 The cpu_baseline leg (N = 1, rank 0) times the CPU oracle (oracle/, test
 infrastructure) over ALL 300 frames of the d2 workload, reports frames/s and
@@ -51,7 +53,7 @@ if ROOT not in sys.path:
 
 METRIC = "HD->SD downscale frames/sec (1/2/4/8 B200) and achieved HBM GB/s vs peak"
 FALLBACK_HBM_GBS = 6650.0  # /opt/skills/guides/B200_PROFILING.md fallback
-ALL_EXTRAS = ("d1", "d3", "d4", "d5", "wide")
+ALL_EXTRAS = ("d1", "d3", "d4", "d5", "wide", "f3")
 
 
 def parse(argv=None):
@@ -635,6 +637,44 @@ def record_wide(aol, peak, check):
     return rec
 
 
+def record_f3(aol, peak, a, frame0, F, d2_cs):
+    """NEXT row f3: the d2 workload through the paper's filters as RUN-TIME descriptors (aol_filter_preset H and V
+    over the stack of planes) chained by aol_filter_chain_apply -- one kernel, specialised at run time
+    by NVRTC for these descriptors (chain_sep.cu).  Parity: every frame's checksum equals the d2 fused kernel's
+    (which the cpu_baseline leg compares with the oracle's for all frames); the two-launch path (Y through HBM) is
+    timed beside it."""
+    import numpy as np
+    import torch
+
+    C, H, W = a.channels, a.H, a.W
+    P = F * C
+    x = aol.synth_frames(a.seed, frame0, F, C, H, W).reshape(P, H, W)
+    fh = aol.filter_preset(aol.FILTER_H, P, H, W)
+    fv = aol.filter_preset(aol.FILTER_V, P, H, 3 * (W // 8))
+    z = torch.empty((P, 4 * (H // 9), 3 * (W // 8)), dtype=torch.int32, device="cuda")
+    aol.filter_chain_apply(fh, fv, x, out=z)   # (first call: run-time compilation)
+    kernel = aol.last_kernel()
+    med, mn = timed(lambda: aol.filter_chain_apply(fh, fv, x, out=z), inner=5)
+    y = torch.empty((P, H, 3 * (W // 8)), dtype=torch.int32, device="cuda")
+    z2 = torch.empty_like(z)
+    med2, _ = timed(lambda: (aol.filter_apply(fh, x, out=y), aol.filter_apply(fv, y, out=z2)), inner=2)
+    cs = aol.frame_checksum(z.reshape(F, C, 4 * (H // 9), 3 * (W // 8)))
+    torch.cuda.synchronize()
+    got = cs.cpu().view(torch.int64).numpy().view(np.uint64)
+    two_equal = bool(torch.equal(z, z2))
+    del x, y, z, z2
+    torch.cuda.empty_cache()
+    b = F * frame_bytes(C, H, W)
+    return {"config": f"f3 the d2 workload ({F} HD frames) through the H and V filters as run-time descriptors, "
+                      "chained in one kernel", "kernel": kernel, "ms": med, "min_ms": mn,
+            "frames_per_s": F / (med / 1e3), "GBps": b / med / 1e6, "frac": b / med / 1e6 / peak,
+            "two_launches_ms": med2, "two_launches_frames_per_s": F / (med2 / 1e3),
+            "two_launches_equal": two_equal, "parity": bool(np.array_equal(got, d2_cs[:F])),
+            "parity_scope": f"all {F} frame checksums equal the d2 fused kernel's (themselves vs the oracle in "
+                            "cpu_baseline)",
+            "timing": "CUDA events, 5 (two launches: 2) calls back to back per event pair, median of 20"}
+
+
 def record_d5(a, aol, world, rank, use_dist, backend, d2_fps_per_gpu, peak, check):
     """configs[4]: the 10,000-frame HD stream frame-sharded across the ranks (strong scaling).
     Rank g owns stream frames [g*T/G, (g+1)*T/G) and cycles them through a device pool of 256 unique frames:
@@ -917,6 +957,8 @@ def main():
             records["d4"] = record_d4(aol, peak, check)
         if "wide" in extras:
             records["wide"] = record_wide(aol, peak, check)
+        if "f3" in extras:
+            records["f3"] = record_f3(aol, peak, a, frame0, F, cs_all)
     if use_dist:
         dist.barrier()
 
