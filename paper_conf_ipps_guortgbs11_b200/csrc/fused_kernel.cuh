@@ -270,6 +270,12 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
     constexpr bool kI32 = std::is_same<Tin, int32_t>::value;
     constexpr bool kIL = !kI32 && kSwz == 3;   // packed 24-bit pixels: a unit covers the 3 planes of a frame
     constexpr bool kStrip = kI32 && kSwz == 1; // column strips (a.segs repetitions each, one row per stage)
+    // Packed pixels stream the unit's halo triple LAST instead of first: its 18 values per thread (rows 9 and 9..11
+    // of the last band, 3 channels x 3 columns) are then consumed at once instead of held in registers through
+    // the unit (the 3-channel consumer spilled at 2 CTAs/SM).  Halo-first makes the halo read coincide with the
+    // neighbouring unit's read of the same rows (an L2 hit) -- what the HBM-bound int32 path needs; this
+    // issue-bound path does not.
+    constexpr bool kHaloLast = kIL;
     constexpr int kC = 3 * kR;                 // Y / Z columns per consumer thread (kIL: 3 channels x 3)
     constexpr int kRP = kIL ? 1 : kR;          // H-tiler repetitions per consumer thread
     extern __shared__ uint8_t smem_raw[];
@@ -317,8 +323,10 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
                 const int64_t row0 = plane * a.H;
                 // halo triple: rows 9*b1 .. 9*b1+2 (mod H -- the V tiler's toroidal wrap for the last band)
                 const int32_t halo = (3 * b1 == a.triples_per_plane) ? 0 : 3 * b1;
+                // (packed pixels load the halo LAST: see kHaloLast)
                 for (int32_t t = 0; t < ntrip; ++t) {
-                    const int32_t trip = t == 0 ? halo : 3 * b0 + t - 1;
+                    const int32_t trip = kHaloLast ? (t == ntrip - 1 ? halo : 3 * b0 + t)
+                                                   : (t == 0 ? halo : 3 * b0 + t - 1);
                     if constexpr (kI32) {
                         if (a.rows_per_stage == 1) {   // one row per stage, three stages per triple
                             for (int32_t q = 0; q < 3; ++q) {
@@ -601,7 +609,7 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
             }
         };
 
-        {   // the halo triple comes first: keep what the unit's last band needs from it (rows 9 and 9..11)
+        if (!kHaloLast) {   // the halo triple comes first: keep what the unit's last band needs (rows 9 and 9..11)
             int32_t y[3][kC];
             triple(y);
 #pragma unroll
@@ -644,6 +652,15 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
                 A1[m] += s2;
                 A2[m] += s2 + y[2][m];
                 A3[m] = s2 + y[2][m];                             // rows 6..8 of window 6..11
+            }
+        }
+        if (kHaloLast) {   // the halo triple now: it completes the unit's last band
+            int32_t y[3][kC];
+            triple(y);
+#pragma unroll
+            for (int m = 0; m < kC; ++m) {
+                Hr9[m] = y[0][m];
+                Hr911[m] = y[0][m] + y[1][m] + y[2][m];
             }
         }
         emit(b1 - 1, Hr9, Hr911);   // the unit's last band, completed by the halo rows
