@@ -433,6 +433,9 @@ def record_d1(aol, peak, check):
     call = lambda: aol.downscale_frame(x, out=z, checksums=cs)  # noqa: E731
     # warm L2: a GPU-side sleep before each call keeps the host enqueue off the device timeline
     warm, _ = timed(call, reps=50, before=lambda: torch.cuda._sleep(200000))
+    # the same measurement of a trivial one-CTA kernel (zeroing 8 bytes): the floor this method can show for ANY
+    # isolated call -- event, launch and completion latency with nothing to do
+    floor, _ = timed(lambda: cs.zero_(), reps=50, before=lambda: torch.cuda._sleep(200000))
     flush = torch.empty(512 << 20, dtype=torch.uint8, device="cuda")   # > 2x the 126 MB L2
     cold, _ = timed(call, reps=50, before=lambda: flush.fill_(1))
     del flush
@@ -492,6 +495,8 @@ def record_d1(aol, peak, check):
     rec = {"config": "d1 single 1920x1080 3-channel frame -> 720x480 (BASELINE configs[0])",
            "warm_l2_us": warm * 1e3, "cold_l2_us": cold * 1e3, "graph_us_per_call": graph_ms * 1e3 / 20,
            "host_enqueue_us_per_call_python": host_us, "roofline_floor_us": b / peak / 1e3,
+           "isolated_call_floor_us": floor * 1e3,
+           "warm_l2_over_floor_us": warm * 1e3 - floor * 1e3,
            "plan": {"warm_l2_us": pwarm * 1e3, "graph_us_per_call": pgraph_ms * 1e3 / 20,
                     "host_enqueue_us_per_call_python": plan_host_us,
                     "host_enqueue_us_per_call_c": c_enq["plan_launch_us"] if c_enq else None,
