@@ -24,12 +24,20 @@ for v in "i32:" "u8:--dtype u8" "u8i16:--dtype u8 --out-dtype i16"; do
       > gpurun_out/${T}_ncu_${name}.log 2>&1
   ncu -i /tmp/ncu/${T}_${name}.ncu-rep --page raw --csv > gpurun_out/${T}_ncu_${name}_raw.csv 2>/dev/null
 done
-timeout 900 ncu --set full --clock-control none -k regex:"tiler|filter" -c 16 \
+timeout 900 ncu --set full --clock-control none -k regex:"tiler|filter" -c 24 \
     -o /tmp/ncu/${T}_tiler -f python tools/tiler_probe_all.py > gpurun_out/${T}_ncu_tiler.log 2>&1
 ncu -i /tmp/ncu/${T}_tiler.ncu-rep --page raw --csv > gpurun_out/${T}_ncu_tiler_raw.csv 2>/dev/null
 timeout 900 ncu --set full --clock-control none -k regex:"chain" -c 1 \
     -o /tmp/ncu/${T}_chain -f python tools/chain_probe.py --ncu > gpurun_out/${T}_ncu_chain.log 2>&1
 ncu -i /tmp/ncu/${T}_chain.ncu-rep --page raw --csv > gpurun_out/${T}_ncu_chain_raw.csv 2>/dev/null
+# the fused kernel's column strips (16 8K DCI frames)
+timeout 900 ncu --set full --clock-control none --import-source on -k regex:fused_tma -s 3 -c 1 \
+    -o /tmp/ncu/${T}_wide -f python bench.py --frames 16 --H 4320 --W 8192 --steps 1 --warmup 3 --no-e2e \
+    --no-cpu-baseline --extras none > gpurun_out/${T}_ncu_wide.log 2>&1
+ncu -i /tmp/ncu/${T}_wide.ncu-rep --page raw --csv > gpurun_out/${T}_ncu_wide_raw.csv 2>/dev/null
+timeout 600 compute-sanitizer --tool racecheck --error-exitcode 3 python tools/sanitize_workload.py --chain-only \
+    > gpurun_out/${T}_sanitize_racecheck_chain.log 2>&1
+echo "racecheck (chain) rc=$?" >> gpurun_out/${T}_sanitize_summary.txt
 for tool in memcheck synccheck; do
   timeout 900 compute-sanitizer --tool $tool --error-exitcode 3 python tools/sanitize_workload.py > gpurun_out/${T}_sanitize_$tool.log 2>&1
   echo "$tool rc=$?" >> gpurun_out/${T}_sanitize_summary.txt

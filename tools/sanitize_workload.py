@@ -21,7 +21,21 @@ def main():
     ap.add_argument("--kernels", default="1,2")
     ap.add_argument("--fused-only", action="store_true")
     ap.add_argument("--widths", default="", help="only these W values, e.g. 256")
+    ap.add_argument("--chain-only", action="store_true", help="only the separable chain kernels (racecheck)")
     args = ap.parse_args()
+    if args.chain_only:   # cp.async row staging + a shared-memory ring behind two barriers per row
+        torch.cuda.set_device(0)
+        P, H, W = 2, 36, 256
+        x = aol.synth_frames(3, 0, 1, P, H, W, "uniform")[0]
+        fh, fv = aol.filter_preset(aol.FILTER_H, P, H, W), aol.filter_preset(aol.FILTER_V, P, H, 3 * W // 8)
+        want = aol.filter_apply(fv, aol.filter_apply(fh, x))
+        ok = True
+        for jit in (1, 0):
+            aol._lib.lib().aol_debug_set_chain_jit(jit)
+            ok &= torch.equal(aol.filter_chain_apply(fh, fv, x), want)
+        torch.cuda.synchronize()
+        print("sanitize workload (chain):", "OK" if ok else "MISMATCH")
+        return 0 if ok else 1
     dts = [{"i32": torch.int32, "u8": torch.uint8}[d] for d in args.dtypes.split(",")]
     kernels = [int(k) for k in args.kernels.split(",")]
     torch.cuda.set_device(0)
@@ -114,6 +128,30 @@ def main():
     Ac = torch.arange(50 * 1000, dtype=torch.int32, device="cuda").reshape(50, 1000)
     tc = aol.make_tiler([50, 1000], [50, 125], [11], [3, -2], [[1, 0], [0, 8]], [[0], [1]])
     aol.tiler_gather(tc, Ac)
+    # round 2, later: the separable chain statically compiled (the default above is the NVRTC-specialised one),
+    # the general chain kernel (V then H), affine pieces with array sides off the 16-byte grid (gather + FAST
+    # scatter, 2 / 4 / 8-byte elements), column strips of the fused kernel (forced at a small width)
+    L = aol._lib.lib()
+    L.aol_debug_set_chain_jit(0)
+    z3 = aol.filter_chain_apply(aol.filter_preset(aol.FILTER_H, P, H, W), aol.filter_preset(aol.FILTER_V, P, H, 3 * W // 8), x)
+    L.aol_debug_set_chain_jit(1)
+    ok &= torch.equal(z, z3)
+    xv = aol.synth_frames(5, 0, 1, 2, 54, 512, "uniform")[0]
+    zvh = aol.filter_chain_apply(aol.filter_preset(aol.FILTER_V, 2, 54, 512), aol.filter_preset(aol.FILTER_H, 2, 24, 512), xv)
+    yv = aol.filter_apply(aol.filter_preset(aol.FILTER_V, 2, 54, 512), xv)
+    ok &= torch.equal(zvh, aol.filter_apply(aol.filter_preset(aol.FILTER_H, 2, 24, 512), yv))
+    for dt in (torch.int16, torch.int32, torch.int64):
+        Ap = torch.arange(3 * 64 * 256, device="cuda").reshape(3, 64, 256).to(dt)
+        tp = aol.make_tiler([3, 64, 256], [3, 8, 32], [8, 8], [0, -3, 5], [[1, 0, 0], [0, 8, 0], [0, 0, 8]], [[0, 0], [1, 0], [0, 1]])
+        Gp = aol.tiler_gather(tp, Ap)
+        Bp = torch.zeros_like(Ap)
+        aol.tiler_scatter(tp, Gp, Bp, mode="fast")
+        ok &= torch.equal(Ap, Bp)
+    xs = aol.synth_frames(6, 0, 2, 3, 27, 1056)
+    zs, css = aol.downscale_frame(xs, checksums=True, opts={"kernel": 1, "flags": aol.FLAGS["I32_STRIPS"]})
+    zt, cst = aol.downscale_frame(xs, checksums=True, opts={"kernel": 2})
+    torch.cuda.synchronize()
+    ok &= torch.equal(zs, zt) and torch.equal(css.view(torch.int64), cst.view(torch.int64))
     xp = aol.synth_frames(4, 0, 2, 3, 36, 256)
     pl = aol.FramePlan(xp, checksums=True)
     zp, csp = pl.launch()
