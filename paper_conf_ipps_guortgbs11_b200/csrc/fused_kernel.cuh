@@ -276,6 +276,12 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
     // neighbouring unit's read of the same rows (an L2 hit) -- what the HBM-bound int32 path needs; this
     // issue-bound path does not.
     constexpr bool kHaloLast = kIL;
+    // 8-bit samples with int16 outputs: outputs stored directly from registers instead of through the smem
+    // staging buffer and a bulk store, whose two CTA barriers per band the issue-bound consumer waited on (HD
+    // uint8 0.416 -> 0.401 ms, packed pixels 0.516 -> 0.479, CIF 0.290 -> 0.284).  int32 outputs keep the bulk
+    // store: direct 8-byte stores cost DRAM efficiency there (uint8 HD 0.481 -> 0.555 ms, packed 0.503 -> 0.511;
+    // profiles/r02_direct_store_ab.jsonl)
+    constexpr bool kDirectStore = !kI32 && sizeof(Tout) == 2;
     constexpr int kC = 3 * kR;                 // Y / Z columns per consumer thread (kIL: 3 channels x 3)
     constexpr int kRP = kIL ? 1 : kR;          // H-tiler repetitions per consumer thread
     extern __shared__ uint8_t smem_raw[];
@@ -479,6 +485,37 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
                     z[3][m] = task_T_small(A3[m] + add911[m]);
                 }
             }
+            if constexpr (kDirectStore) {
+                // each thread stores its outputs straight to Z from registers (per plane and row: its 3 kR columns
+                // at column 3r, coalesced across the warp in the widest aligned words) -- no staging, no barriers
+                if (active) {
+                    constexpr int kPl = kIL ? 3 : 1;       // planes per unit
+                    constexpr int kCols = kC / kPl;        // columns per plane and row: 3 kR (or 3)
+#pragma unroll
+                    for (int j = 0; j < kPl; ++j) {
+                        Tout* gz = static_cast<Tout*>(a.Z) +
+                                   (size_t(kPl * plane + j) * a.Ho + size_t(4 * band)) * size_t(Wo) + 3 * r;
+#pragma unroll
+                        for (int k = 0; k < 4; ++k) {
+                            Tout* row = gz + size_t(k) * Wo;
+                            const int32_t* v = &z[k][kCols * j];
+                            if constexpr (sizeof(Tout) == 2 && kCols % 2 == 0) {   // 12 r bytes: 4-byte words
+#pragma unroll
+                                for (int m = 0; m < kCols; m += 2)
+                                    reinterpret_cast<uint32_t*>(row)[m / 2] =
+                                        __byte_perm(uint32_t(v[m]), uint32_t(v[m + 1]), 0x5410u);
+                            } else if constexpr (sizeof(Tout) == 4 && kCols % 2 == 0) {   // 24 tid bytes: 8-byte words
+#pragma unroll
+                                for (int m = 0; m < kCols; m += 2)
+                                    reinterpret_cast<int2*>(row)[m / 2] = make_int2(v[m], v[m + 1]);
+                            } else {
+#pragma unroll
+                                for (int m = 0; m < kCols; ++m) row[m] = Tout(v[m]);
+                            }
+                        }
+                    }
+                }
+            } else {
             if (tid == 0) ptx::bulk_wait_read<kOutBufs - 1>();   // the out buffer we reuse is free again
             ptx::named_bar_sync(1, NC);
             const uint32_t ob = ptx::smem_u32(outbuf) + (emit_idx % kOutBufs) * a.out_bytes;
@@ -543,6 +580,7 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
                 ptx::bulk_store(gz, src, a.out_bytes);   // 4 rows
                 ptx::bulk_commit();
             }
+            }   // !kDirectStore
             ++emit_idx;
             if constexpr (kChecksum && kIL) {
               if (active) {
