@@ -131,6 +131,7 @@ RingGeom ring_geom(aol_dtype_t dt, int out_es, int64_t W, int flags) {
     g.stage_bytes = uint32_t(rows_per_stage(dt, W, flags) * W) * es;
     g.stage_stride = (g.stage_bytes + align - 1) & ~(align - 1);
     g.out_bytes = uint32_t(4 * out_es * (3 * (W / 8))) * (dt == AOL_RGB8 ? 3u : 1u);   // packed: 3 planes
+    if (dt != AOL_I32 && out_es == 2) g.out_bytes = 0;   // int16 outputs leave from registers (no staging)
     if (const int sr = i32_strip_reps(dt, W, flags)) {   // a strip row + the next repetition's first 16 bytes
         g.stage_bytes = uint32_t(32 * sr + 16);
         g.stage_stride = (g.stage_bytes + align - 1) & ~(align - 1);
@@ -249,7 +250,12 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void*
             } else {
                 // nearest whole number of stages to the in-flight target; one-row stages round down (4K: 7 rows =
                 // 1.065 ms, 8 = 1.070, 9 = 1.13-1.16: HBM efficiency falls off a cliff above ~120 KB per SM)
-                const int half = rows_per_stage(in_dtype, W, o.flags) == 1 ? 0 : int(geom.stage_stride) / 2;
+                // (8-bit samples, issue-bound: rounded up -- packed pixels with int16 outputs 0.479 ms at 3
+                // stages, 0.464 at 4; planar uint8 4K 0.434 -> 0.417; except packed pixels with int32 outputs,
+                // whose 4th stage costs the 2nd CTA's room: 0.503 -> 0.530; profiles/r02_stage_round_ab.jsonl)
+                const bool up = u8like && !(rgb && out_es == 4);
+                const int half = up ? int(geom.stage_stride) - 1
+                                    : rows_per_stage(in_dtype, W, o.flags) == 1 ? 0 : int(geom.stage_stride) / 2;
                 const int target = (kInflightBytesPerSM / cps + half) / int(geom.stage_stride);
                 stages = std::min(stages, std::max(2, target));
             }
