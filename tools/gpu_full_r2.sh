@@ -1,6 +1,6 @@
 #!/bin/bash
 # round 2 full run: every GPU test, smoke, the default bench (all records), variants, reference arm,
-# ncu launch list + full captures (headline i32, u8, u8->i16, every tiler / filter / chain kernel), sanitizers
+# ncu launch list + full captures (headline i32, u8, u8->i16, every tiler / filter / chain kernel), sanitizer workload
 cd "$GRAFT_REPO_ROOT"
 mkdir -p gpurun_out
 T=${TAG:-r02_full}
@@ -35,10 +35,7 @@ timeout 900 ncu --set full --clock-control none --import-source on -k regex:fuse
     -o /tmp/ncu/${T}_wide -f python bench.py --frames 16 --H 4320 --W 8192 --steps 1 --warmup 3 --no-e2e \
     --no-cpu-baseline --extras none > gpurun_out/${T}_ncu_wide.log 2>&1
 ncu -i /tmp/ncu/${T}_wide.ncu-rep --page raw --csv > gpurun_out/${T}_ncu_wide_raw.csv 2>/dev/null
-timeout 600 compute-sanitizer --tool racecheck --error-exitcode 3 python tools/sanitize_workload.py --chain-only \
-    > gpurun_out/${T}_sanitize_racecheck_chain.log 2>&1
-echo "racecheck (chain) rc=$?" >> gpurun_out/${T}_sanitize_summary.txt
-for tool in memcheck synccheck; do
-  timeout 900 compute-sanitizer --tool $tool --error-exitcode 3 python tools/sanitize_workload.py > gpurun_out/${T}_sanitize_$tool.log 2>&1
-  echo "$tool rc=$?" >> gpurun_out/${T}_sanitize_summary.txt
-done
+# compute-sanitizer is closed on the GPU pool (runs under it left GPUs needing a reset): the sanitizer workload
+# runs directly (every kernel on small shapes, cross-path agreement asserted)
+timeout 600 python tools/sanitize_workload.py > gpurun_out/${T}_sanitize_workload.log 2>&1
+echo "sanitize workload (no sanitizer) rc=$?" >> gpurun_out/${T}_sanitize_summary.txt
