@@ -233,12 +233,13 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void*
         // concurrent row streams than that: DRAM efficiency falls as streams are added.  int32
         // (HBM-bound): 8 consumer warps per SM.  uint8 (issue-bound): 16 warps of one repetition each,
         // or 8 warps of two (HD: 2 CTAs/SM, 0.499 ms vs 0.567 at 3 and 0.738 at 1;
-        // profiles/r01_u8_r2_ab.jsonl) -- 12 with int16 outputs, whose halved write traffic leaves DRAM room
-        // for a third row stream per SM (HD: 0.431 ms at 3 CTAs/SM vs 0.503 at 2; profiles/r01_u8_i16.jsonl).
+        // profiles/r01_u8_r2_ab.jsonl) -- 16 with int16 outputs, whose halved write traffic leaves DRAM room
+        // for more row streams per SM (HD: 0.431 ms at 3 CTAs/SM vs 0.503 at 2, profiles/r01_u8_i16.jsonl; 0.397
+        // at 4 with the 96-register instantiation, profiles/r02_u8_cps4_ab.jsonl).
         const int cwarps = nc / 32;
         // packed 24-bit pixels (3 channels per thread, ~100 registers): 16 warps (HD: 2 CTAs/SM 0.513 ms vs 0.608
         // at 1; profiles/r01_rgb_sweep.jsonl)
-        const int want_warps = rgb ? 16 : (in_dtype == AOL_U8 && kr == 1) ? 16 : (in_dtype == AOL_U8 && out_es == 2) ? 12 : 8;
+        const int want_warps = rgb ? 16 : (in_dtype == AOL_U8 && (kr == 1 || out_es == 2)) ? 16 : 8;
         cps = o.ctas_per_sm > 0 ? o.ctas_per_sm
                                 : std::max(1, std::min(8, (want_warps + cwarps - 1) / cwarps));
         for (;; --cps) {

@@ -33,6 +33,7 @@ def test_bench_default_contract():
     assert r["bound"] == "hbm" and r["unit"] == "GB/s" and abs(r["frac"] - r["achieved"] / r["peak"]) < 1e-9
     assert {"value", "unit", "h2d_bytes_per_step", "d2h_bytes_per_step"} <= set(d["e2e"])
     assert d["e2e"]["checksums_match_device_path"] is True
+    assert 0.0 < d["e2e"]["frac_of_h2d_probe"] < 1.5
     cb = d["cpu_baseline"]
     assert cb["kind"] == "oracle" and cb["parity_all_frames"] is True and cb["frames_compared"] == 12
     assert cb["GBps_algorithmic"] > 0 and cb["cores"] >= 1
