@@ -27,7 +27,10 @@ frames), d5 (the 10,000-frame stream frame-sharded over the N ranks: strong
 scaling, at every N; every stream frame's checksum verified), wide (16 8K DCI
 frames, 8192 wide: the fused kernel's column strips), f3 (the same 300 frames
 through the paper's H and V filters as run-time descriptors, chained into one
-kernel specialised at run time; its checksums must equal the d2 kernel's).
+kernel specialised at run time; its checksums must equal the d2 kernel's), f1 (the
+same frames as 8-bit samples, planar and packed 24-bit pixels, int32 and int16
+outputs; checksums equal the d2 kernel's), f4 (2000 CIF frames, all checksums vs
+the oracle).
 
 The cpu_baseline leg (N = 1, rank 0) times the CPU oracle (oracle/, test
 infrastructure) over ALL 300 frames of the d2 workload, reports frames/s and
@@ -53,7 +56,7 @@ if ROOT not in sys.path:
 
 METRIC = "HD->SD downscale frames/sec (1/2/4/8 B200) and achieved HBM GB/s vs peak"
 FALLBACK_HBM_GBS = 6650.0  # /opt/skills/guides/B200_PROFILING.md fallback
-ALL_EXTRAS = ("d1", "d3", "d4", "d5", "wide", "f3")
+ALL_EXTRAS = ("d1", "d3", "d4", "d5", "wide", "f1", "f3", "f4")
 
 
 def parse(argv=None):
@@ -680,6 +683,84 @@ def record_f3(aol, peak, a, frame0, F, d2_cs):
             "timing": "CUDA events, 5 (two launches: 2) calls back to back per event pair, median of 20"}
 
 
+def record_f1(aol, peak, a, frame0, F, d2_cs):
+    """NEXT row f1: the d2 workload's frames stored as 8-bit samples (P:L260's 24-bit RGB) -- planar uint8 planes
+    and packed [N][H][W][3] pixels (OpenCV's layout), each with int32 and int16 outputs.  The samples
+    are the same integers as the d2 int32 input, so every frame's checksum must equal the d2 kernel's (itself
+    compared with the oracle for all frames in cpu_baseline).  Each variant's `mix_frac` is its time against the
+    HBM probe's best rate for its own read:write byte mix (the 8-bit paths are issue-bound, not HBM-bound)."""
+    import numpy as np
+    import torch
+
+    C, H, W = a.channels, a.H, a.W
+    Ho, Wo = 4 * (H // 9), 3 * (W // 8)
+    x8 = aol.synth_frames(a.seed, frame0, F, C, H, W, "uniform", dtype=torch.uint8)
+    xp = x8.permute(0, 2, 3, 1).contiguous()   # packed 24-bit pixels [F][H][W][3]
+    recs = []
+    for layout, xin, fn in (("planar uint8", x8, aol.downscale_frame),
+                            ("packed 24-bit pixels", xp, aol.downscale_frame_packed)):
+        for odt, oname in ((torch.int32, "int32"), (torch.int16, "int16")):
+            z = torch.empty((F, C, Ho, Wo), dtype=odt, device="cuda")
+            cs = torch.empty(F, dtype=torch.uint64, device="cuda")
+            with ClockSampler(torch.cuda.current_device()) as clk:
+                med, mn = timed(lambda: fn(xin, out=z, checksums=cs), inner=5)
+                # the headline's method as well: 50 calls back to back between one event pair
+                e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+                e0.record()
+                for _ in range(50):
+                    fn(xin, out=z, checksums=cs)
+                e1.record()
+                torch.cuda.synchronize()
+                run_ms = e0.elapsed_time(e1) / 50
+            got = cs.cpu().view(torch.int64).numpy().view(np.uint64)
+            b = F * frame_bytes(C, H, W, es=1, eo=odt.itemsize)
+            mix, _ = mix_ceiling(argparse.Namespace(dtype="u8", out_dtype="i16" if odt == torch.int16 else "i32"))
+            recs.append({"config": f"f1 {F} HD frames, {layout} -> {oname} outputs", "ms": med, "min_ms": mn,
+                         "frames_per_s": F / (med / 1e3), "GBps": b / med / 1e6, "frac": b / med / 1e6 / peak,
+                         "mix_ceiling_GBps": mix, "mix_frac": (b / med / 1e6 / mix) if mix else None,
+                         "plan": aol.downscale_frame_plan(F, C, H, W, out_dtype=odt,
+                                                          dtype="rgb8" if layout.startswith("packed") else torch.uint8),
+                         "parity": bool(np.array_equal(got, d2_cs[:F])),
+                         "parity_scope": f"all {F} frame checksums equal the d2 kernel's (themselves vs the oracle "
+                                         "in cpu_baseline)",
+                         "ms_50_back_to_back": run_ms, "clocks": clk.summary(),
+                         "timing": "CUDA events, 5 calls back to back per event pair, median of 20"})
+            del z, cs
+    del x8, xp
+    torch.cuda.empty_cache()
+    return recs
+
+
+def record_f4(aol, peak, check):
+    """NEXT row f4: the paper's second workload (Section III): 2000 CIF frames 352x288x3 -> 132x128x3
+    in one launch (int32); all 2000 checksums against the oracle."""
+    import numpy as np
+    import torch
+
+    N, C, H, W, seed = 2000, 3, 288, 352, 3
+    x = aol.synth_frames(seed, 0, N, C, H, W)
+    z = torch.empty((N, C, 4 * (H // 9), 3 * (W // 8)), dtype=torch.int32, device="cuda")
+    cs = torch.empty(N, dtype=torch.uint64, device="cuda")
+    med, mn = timed(lambda: aol.downscale_frame(x, out=z, checksums=cs), inner=5)
+    b = N * frame_bytes(C, H, W)
+    mix, _ = mix_ceiling(argparse.Namespace(dtype="i32", out_dtype="i32"))
+    rec = {"config": "f4 2000 CIF frames 352x288x3 int32 -> 132x128x3 (Section III's second workload)", "ms": med,
+           "min_ms": mn, "frames_per_s": N / (med / 1e3), "GBps": b / med / 1e6, "frac": b / med / 1e6 / peak,
+           "mix_frac": (b / med / 1e6 / mix) if mix else None,
+           "timing": "CUDA events, 5 calls back to back per event pair, median of 20",
+           "plan": aol.downscale_frame_plan(N, C, H, W)}
+    torch.cuda.synchronize()
+    got = cs.cpu().view(torch.int64).numpy().view(np.uint64)
+    del x, z, cs
+    torch.cuda.empty_cache()
+    if check:
+        ref, spent = oracle_checksums(seed, range(N), C, H, W, oracle_threads())
+        rec["parity"] = bool(np.array_equal(ref, got))
+        rec["parity_scope"] = f"all {N} frame checksums vs the oracle"
+        rec["cpu_oracle_frames_per_s"] = N / spent
+    return rec
+
+
 def record_d5(a, aol, world, rank, use_dist, backend, d2_fps_per_gpu, peak, check):
     """configs[4]: the 10,000-frame HD stream frame-sharded across the ranks (strong scaling).
     Rank g owns stream frames [g*T/G, (g+1)*T/G) and cycles them through a device pool of 256 unique frames:
@@ -979,8 +1060,12 @@ def main():
             records["d4"] = record_d4(aol, peak, check)
         if "wide" in extras:
             records["wide"] = record_wide(aol, peak, check)
+        if "f1" in extras:
+            records["f1"] = record_f1(aol, peak, a, frame0, F, cs_all)
         if "f3" in extras:
             records["f3"] = record_f3(aol, peak, a, frame0, F, cs_all)
+        if "f4" in extras:
+            records["f4"] = record_f4(aol, peak, check)
     if use_dist:
         dist.barrier()
 

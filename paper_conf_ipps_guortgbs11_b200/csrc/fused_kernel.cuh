@@ -276,14 +276,15 @@ __global__ void __launch_bounds__(kMaxThreads, kMinBlocks)
     // store: direct 8-byte stores cost DRAM efficiency there (uint8 HD 0.481 -> 0.555 ms, packed 0.503 -> 0.511;
     // profiles/r02_direct_store_ab.jsonl)
     constexpr bool kDirectStore = !kI32 && sizeof(Tout) == 2;
-    // Packed pixels, and planar 8-bit samples with two repetitions per thread at 4 CTAs/SM (int16 outputs), stream
-    // the unit's halo triple LAST instead of first: its values (rows 9 and 9..11 of the last band) are then
-    // consumed at once instead of held in registers through the unit -- the 3-channel consumer spilled at 2
-    // CTAs/SM, and the planar one fits the 102-register budget of 4 CTAs/SM without spills only this way (HD
-    // uint8 -> int16 0.403 -> 0.397 ms; halo-last at 3 CTAs/SM, or for int32 outputs, CIF and 4K: no gain or up to
-    // 3 % slower; profiles/r02_u8_cps4_ab.jsonl).  Halo-first makes the halo read coincide with the neighbouring
-    // unit's read of the same rows (an L2 hit) -- what the HBM-bound paths need; these issue-bound ones do not.
-    constexpr bool kHaloLast = kIL || (kDirectStore && kR == 2 && kMinBlocks >= 4);
+    // Packed pixels, and planar 8-bit samples with two repetitions per thread in the multi-CTA int16-output
+    // instantiations (HD: 4 CTAs/SM of 160 threads; 4K: 2 of 288), stream the unit's halo triple LAST instead of
+    // first: its values (rows 9 and 9..11 of the last band) are then consumed at once instead of held in
+    // registers through the unit -- the 3-channel consumer spilled at 2 CTAs/SM, and the planar one fits 96
+    // registers without spills only this way (HD uint8 -> int16 0.403 -> 0.395 ms at 4 CTAs/SM, 4K 0.362 ->
+    // 0.343 at 2; halo-last at 3 CTAs/SM, or for int32 outputs and CIF: no gain or up to 3 % slower;
+    // profiles/r02_u8_cps4_ab.jsonl, profiles/r02_u8_4k_cps2_ab.jsonl).  Halo-first makes the halo read coincide
+    // with the neighbouring unit's read of the same rows (an L2 hit) -- what the HBM-bound paths need.
+    constexpr bool kHaloLast = kIL || (kDirectStore && kR == 2 && kMinBlocks * kMaxThreads >= 576);
     constexpr int kC = 3 * kR;                 // Y / Z columns per consumer thread (kIL: 3 channels x 3)
     constexpr int kRP = kIL ? 1 : kR;          // H-tiler repetitions per consumer thread
     extern __shared__ uint8_t smem_raw[];
@@ -838,9 +839,12 @@ KernelFn pick_tma_kernel(int block, int cps) {
         return fused_tma_kernel<Tin, Tout, kR, kSwz, kChecksum, 1024, 1>;
     } else if constexpr (kR == 2) {
         // two repetitions per thread take ~126 registers: bounds that never force spills below 1024 threads
-        // int16 outputs at 4 CTAs/SM: 96 registers, no spills with the halo triple streamed last (see kHaloLast)
-        if constexpr (std::is_same<Tout, int16_t>::value)
+        // int16 outputs at 4 CTAs/SM (HD) / 2 CTAs/SM (4K): 96 registers, no spills with the halo triple streamed
+        // last (see kHaloLast)
+        if constexpr (std::is_same<Tout, int16_t>::value) {
             if (block <= 160 && cps >= 4) return fused_tma_kernel<Tin, Tout, kR, kSwz, kChecksum, 160, 4>;
+            if (block > 256 && block <= 288 && cps >= 2) return fused_tma_kernel<Tin, Tout, kR, kSwz, kChecksum, 288, 2>;
+        }
         if (block <= 160 && cps >= 3) return fused_tma_kernel<Tin, Tout, kR, kSwz, kChecksum, 160, 3>;
         if (block <= 256 && cps >= 2) return fused_tma_kernel<Tin, Tout, kR, kSwz, kChecksum, 256, 2>;
         if (block <= 512) return fused_tma_kernel<Tin, Tout, kR, kSwz, kChecksum, 512, 1>;

@@ -14,12 +14,12 @@ import bench  # noqa: E402
 
 
 def test_extras_selection():
-    assert bench.extras_of(bench.parse([])) == ["d1", "d3", "d4", "d5", "wide", "f3"]
+    assert bench.extras_of(bench.parse([])) == ["d1", "d3", "d4", "d5", "wide", "f1", "f3", "f4"]
     assert bench.extras_of(bench.parse(["--H", "36", "--W", "128"])) == []
     assert bench.extras_of(bench.parse(["--dtype", "u8"])) == []
     assert bench.extras_of(bench.parse(["--extras", "d1,d5"])) == ["d1", "d5"]
     assert bench.extras_of(bench.parse(["--extras", "none"])) == []
-    assert bench.extras_of(bench.parse(["--H", "36", "--extras", "all"])) == ["d1", "d3", "d4", "d5", "wide", "f3"]
+    assert bench.extras_of(bench.parse(["--H", "36", "--extras", "all"])) == ["d1", "d3", "d4", "d5", "wide", "f1", "f3", "f4"]
 
 
 def test_src_hash_and_stale_capture_guard(tmp_path, monkeypatch):

@@ -57,11 +57,13 @@ def test_bench_full_default_run_records_and_parity():
     cb = d["cpu_baseline"]
     assert cb["parity_all_frames"] is True and cb["frames_compared"] == 300
     rec = d["records"]
-    assert set(rec) == {"d1", "d3", "d4", "d5", "wide", "f3"}
+    assert set(rec) == {"d1", "d3", "d4", "d5", "wide", "f1", "f3", "f4"}
     assert rec["d1"]["parity"] is True and rec["d1"]["graph_us_per_call"] > 0
     assert len(rec["d3"]) == 3 and all(r["parity"] is True for r in rec["d3"])
     assert rec["d4"]["parity"] is True and rec["d4"]["frames_per_s"] > 10000
     assert rec["wide"]["parity"] is True and rec["wide"]["kernel"] == "fused_tma_kernel"
     assert rec["f3"]["parity"] is True and rec["f3"]["two_launches_equal"] is True
+    assert len(rec["f1"]) == 4 and all(r["parity"] is True for r in rec["f1"])
+    assert rec["f4"]["parity"] is True and rec["f4"]["frames_per_s"] > 100000
     assert rec["d5"]["parity"] is True and rec["d5"]["scaling"] == "strong" and rec["d5"]["n_gpus"] == 1
     assert d["parity_all_records"] is True
