@@ -101,6 +101,21 @@ bool sep_tiler(const aol_tiler_t& t, int n, int64_t pav_row, int64_t pav_col, in
     return true;
 }
 
+// Bands of f2 per work unit: up to `cap` (a unit re-reads L2 - p2 rows of its neighbour: 3 of every 9 nb rows for
+// the paper's V filter), fewer when that leaves fewer than 4 units per SM.  AOL_SEP_BANDS overrides the cap (A/B).
+void sep_set_bands(SepDev* sd, int cap, const DeviceInfo& dev) {
+    static const int forced = [] {
+        const char* e = std::getenv("AOL_SEP_BANDS");
+        return e ? std::atoi(e) : 0;
+    }();
+    if (forced >= 1) cap = forced;
+    int64_t nb = std::min<int64_t>(cap, sd->R2);
+    while (nb > 1 && int64_t(sd->planes) * ((sd->R2 + nb - 1) / nb) < int64_t(dev.num_sms) * 4) --nb;
+    sd->nb = int32_t(nb);
+    sd->runs = int32_t((sd->R2 + nb - 1) / nb);
+    sd->nunits = int32_t(int64_t(sd->planes) * sd->runs);
+}
+
 // Recognise the separable chain and fill the kernel descriptor; false (why set) when it does not apply.
 bool plan_sep(const aol_filter_t* f1, const aol_filter_t* f2, const DeviceInfo& dev, SepDev* sd, int* smem,
               const char** why) {
@@ -175,13 +190,8 @@ bool plan_sep(const aol_filter_t* f1, const aol_filter_t* f2, const DeviceInfo& 
         return false;
     }
     *smem = int(bytes);
-    // bands per unit: 8 (the run re-reads L2 - p2 rows of its neighbour: 4 % for the paper's V filter), fewer
-    // when that leaves fewer than 4 units per SM
-    int64_t nb = std::min<int64_t>(8, R2);
-    while (nb > 1 && planes * ((R2 + nb - 1) / nb) < int64_t(dev.num_sms) * 4) --nb;
-    sd->nb = int32_t(nb);
-    sd->runs = int32_t((R2 + nb - 1) / nb);
-    sd->nunits = int32_t(planes * sd->runs);
+    sd->planes = int32_t(planes);
+    sep_set_bands(sd, 8, dev);
     return true;
 }
 
@@ -226,6 +236,28 @@ const Nvrtc& nvrtc() {
     return n;
 }
 
+// f1 repetitions per thread of the register-resident column filter (sep_reg_body), 0 when it does not apply: at
+// most two repetitions per thread and 64 accumulators (AOL_SEP_REG=0 keeps the Y ring, for A/B measurements).
+int sep_reg_rpt(const SepDev& sd) {
+    static const bool enabled = [] {
+        const char* e = std::getenv("AOL_SEP_REG");
+        return !(e && e[0] == '0');
+    }();
+    const int rpt = (sd.R1 + kSepThreads - 1) / kSepThreads;
+    const int nbl = (sd.L2 + sd.p2 - 1) / sd.p2;
+    return enabled && rpt <= 2 && nbl * sd.nw2 * sd.nw1 * rpt <= 64 ? rpt : 0;
+}
+
+// X row buffers of the register-resident kernel (AOL_SEP_NBUF overrides, for A/B measurements)
+int sep_reg_nbuf() {
+    static const int n = [] {
+        const char* e = std::getenv("AOL_SEP_NBUF");
+        const int v = e ? std::atoi(e) : 0;
+        return v >= 2 && v <= 16 ? v : 3;   // 3: 1.358 ms vs 1.364 at 4, 1.51 at 5-6 (profiles/r02_f3_reg_sweep.jsonl)
+    }();
+    return n;
+}
+
 // The literal parameters the specialised kernel is compiled for (also its cache key): the filters' patterns,
 // windows and divisors, and the array shapes (a video's frame size is fixed; a new one compiles once more).
 std::string sep_preamble(const aol_filter_t* f1, const aol_filter_t* f2, const SepDev& sd) {
@@ -242,6 +274,10 @@ std::string sep_preamble(const aol_filter_t* f1, const aol_filter_t* f2, const S
                   "#define SEP_R1 %d\n#define SEP_J %d\n#define SEP_XSTRIDE %d\n#define SEP_VEC %d\n#define SEP_O1C %d\n",
                   sd.HX, sd.WX, sd.HY, sd.WY, sd.HZ, sd.R1, sd.J, sd.xstride, sd.vec, sd.o1c);
     s += b;
+    if (const int rpt = sep_reg_rpt(sd)) {
+        std::snprintf(b, sizeof b, "#define SEP_REG 1\n#define SEP_RPT %d\n#define SEP_NBUF %d\n", rpt, sep_reg_nbuf());
+        s += b;
+    }
     for (int f = 0; f < 2; ++f) {
         const aol_filter_t* fl = f == 0 ? f1 : f2;
         const int L = f == 0 ? sd.L1 : sd.L2;
@@ -341,6 +377,10 @@ bool launch_sep_chain(const aol_filter_t* f1, const aol_filter_t* f2, const int3
     const void* jit = sep_jit_kernel(f1, f2, sd);
     const void* kern = jit ? jit : reinterpret_cast<const void*>(sep_kernel_for(sd.L1, sd.L2));
     const char* name = jit ? "sep_chain_jit" : "sep_chain_kernel";
+    if (jit && sep_reg_rpt(sd)) {
+        smem = int(4 * int64_t(sep_reg_nbuf()) * sd.xstride);   // no Y ring
+        sep_set_bands(&sd, 24, dev);   // longer units: 1.358 ms at 24 bands vs 1.386 at 16 and 1.440 at 8
+    }
     *st = kernel_smem(kern, smem);
     if (*st != AOL_OK) return true;
     const int per_sm = std::max(1, kernel_occupancy(kern, kSepThreads, smem));

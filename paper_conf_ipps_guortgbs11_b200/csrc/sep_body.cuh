@@ -25,7 +25,7 @@ struct SepDev {
     sep_i32 p2, L2, nw2, o2r, R2;
     sep_i32 d1, d2;
     sep_u32 d1_mul, d1_sh, d2_mul, d2_sh;
-    sep_i32 nb, runs, nunits;
+    sep_i32 nb, runs, nunits, planes;
     sep_i32 J, xstride, vec;   // staged row length, buffer stride (elements), 16-byte staging
     sep_i32 m1[kSepNW][kSepNP], m2[kSepNW][kSepNP];   // window masks (0/1)
 };
@@ -110,6 +110,68 @@ __device__ __forceinline__ sep_u32 sep_smem_u32(const void* p) {
     return sep_u32(__cvta_generic_to_shared(p));
 }
 
+// f1's pattern of repetition q from the staged X row (the row starts at column o1c, so repetition q's pattern
+// is elements p1 q .. p1 q + NP1 - 1; elements past L1 are masked out by the window masks).
+template <int NP1>
+__device__ __forceinline__ void sep_load_pattern(const SepDev& sd, const sep_i32* xr, sep_i32 q, int tid,
+                                                 sep_i32 (&x)[NP1]) {
+    (void)sd;
+    const sep_i32* xp = xr + SEP_P1 * q;
+    if (NP1 % 4 == 0 && SEP_P1 % 4 == 0) {
+        // 16-byte aligned pattern: NP1/4 LDS.128 (scalar loads at a stride of p1 words conflict p1/gcd-way on the
+        // banks).  At p1 = 8 a quarter-warp's chunks v sit in every other 16-byte bank group: lanes with bit 2 set
+        // take chunks 0 and 1 in the other order, which spreads both loads over all 8 groups (conflict-free).
+        const bool swp = SEP_P1 == 8 && ((tid >> 2) & 1);
+        const int4* xp4 = reinterpret_cast<const int4*>(xp);
+        int4 c[NP1 / 4 > 0 ? NP1 / 4 : 1];
+#pragma unroll
+        for (int v = 0; v < NP1 / 4; ++v) c[v] = xp4[v];
+        if (NP1 >= 8) {
+            const int4 L0 = xp4[swp ? 1 : 0], L1 = xp4[swp ? 0 : 1];   // load slots 0 and 1
+            c[0] = swp ? L1 : L0;
+            c[1] = swp ? L0 : L1;
+        }
+#pragma unroll
+        for (int v = 0; v < NP1 / 4; ++v) {
+            x[4 * v] = c[v].x;
+            x[4 * v + 1] = c[v].y;
+            x[4 * v + 2] = c[v].z;
+            x[4 * v + 3] = c[v].w;
+        }
+    } else {
+#pragma unroll
+        for (int p = 0; p < NP1; ++p) x[p] = xp[p];
+    }
+}
+
+// Stage one X row in shared memory: J elements from column o1c on (mod WX), by cp.async (16-byte chunks when the
+// column origin and width allow).  (sd is only read by the static kernel: the JIT one has every parameter as a
+// literal.)
+__device__ __forceinline__ void sep_stage_row(const SepDev& sd, const sep_i32* src, sep_u32 dst, int tid) {
+    (void)sd;
+    // (one conditional subtraction when the staged span wraps at most once, o1c + J <= 2 WX)
+    const bool once = SEP_O1C + SEP_J <= 2 * SEP_WX;
+    if (SEP_VEC) {   // o1c, WX multiples of 4: every 16-byte chunk lies on one side of the wrap
+        for (sep_i32 c = tid; 4 * c < SEP_J; c += kSepThreads) {
+            sep_i32 col = SEP_O1C + 4 * c;
+            if (once)
+                col -= col >= SEP_WX ? SEP_WX : 0;
+            else
+                while (col >= SEP_WX) col -= SEP_WX;
+            sep_cp_async16(dst + 16u * sep_u32(c), src + col);
+        }
+    } else {
+        for (sep_i32 e = tid; e < SEP_J; e += kSepThreads) {
+            sep_i32 col = SEP_O1C + e;
+            if (once)
+                col -= col >= SEP_WX ? SEP_WX : 0;
+            else
+                while (col >= SEP_WX) col -= SEP_WX;
+            sep_cp_async4(dst + 4u * sep_u32(e), src + col);
+        }
+    }
+}
+
 template <int NP1, int NP2>
 __device__ __forceinline__ void sep_chain_body(const SepDev& sd, const sep_i32* __restrict__ X,
                                                sep_i32* __restrict__ Z, sep_i32* sm) {
@@ -131,27 +193,7 @@ __device__ __forceinline__ void sep_chain_body(const SepDev& sd, const sep_i32* 
             if (staged < nrows) {
                 const sep_i32* src = Xp + sep_i64(xrow_next) * SEP_WX;
                 const sep_u32 dst = sep_smem_u32(xb + (staged % kSepNB) * SEP_XSTRIDE);
-                // (one conditional subtraction when the staged span wraps at most once, o1c + J <= 2 WX)
-                const bool once = SEP_O1C + SEP_J <= 2 * SEP_WX;
-                if (SEP_VEC) {   // o1c, WX multiples of 4: every 16-byte chunk lies on one side of the wrap
-                    for (sep_i32 c = tid; 4 * c < SEP_J; c += kSepThreads) {
-                        sep_i32 col = SEP_O1C + 4 * c;
-                        if (once)
-                            col -= col >= SEP_WX ? SEP_WX : 0;
-                        else
-                            while (col >= SEP_WX) col -= SEP_WX;
-                        sep_cp_async16(dst + 16u * sep_u32(c), src + col);
-                    }
-                } else {
-                    for (sep_i32 e = tid; e < SEP_J; e += kSepThreads) {
-                        sep_i32 col = SEP_O1C + e;
-                        if (once)
-                            col -= col >= SEP_WX ? SEP_WX : 0;
-                        else
-                            while (col >= SEP_WX) col -= SEP_WX;
-                        sep_cp_async4(dst + 4u * sep_u32(e), src + col);
-                    }
-                }
+                sep_stage_row(sd, src, dst, tid);
                 ++staged;
                 if (++xrow_next == SEP_HX) xrow_next = 0;   // Y rows (and so X rows) advance by one, toroidally
             }
@@ -172,33 +214,7 @@ __device__ __forceinline__ void sep_chain_body(const SepDev& sd, const sep_i32* 
                 sep_i32* yr = ring + yslot * SEP_WY;
                 for (sep_i32 q = tid; q < SEP_R1; q += kSepThreads) {
                     sep_i32 x[NP1];
-                    const sep_i32* xp = xr + SEP_P1 * q;
-                    if (NP1 % 4 == 0 && SEP_P1 % 4 == 0) {
-                        // 16-byte aligned pattern: NP1/4 LDS.128 (scalar loads at a stride of p1 words conflict
-                        // p1/gcd-way on the banks).  At p1 = 8 a quarter-warp's chunks v sit in every other
-                        // 16-byte bank group: lanes with bit 2 set take chunks 0 and 1 in the other order, which
-                        // spreads both loads over all 8 groups (conflict-free).
-                        const bool swp = SEP_P1 == 8 && ((tid >> 2) & 1);
-                        const int4* xp4 = reinterpret_cast<const int4*>(xp);
-                        int4 c[NP1 / 4 > 0 ? NP1 / 4 : 1];
-#pragma unroll
-                        for (int v = 0; v < NP1 / 4; ++v) c[v] = xp4[v];
-                        if (NP1 >= 8) {
-                            const int4 L0 = xp4[swp ? 1 : 0], L1 = xp4[swp ? 0 : 1];   // load slots 0 and 1
-                            c[0] = swp ? L1 : L0;
-                            c[1] = swp ? L0 : L1;
-                        }
-#pragma unroll
-                        for (int v = 0; v < NP1 / 4; ++v) {
-                            x[4 * v] = c[v].x;
-                            x[4 * v + 1] = c[v].y;
-                            x[4 * v + 2] = c[v].z;
-                            x[4 * v + 3] = c[v].w;
-                        }
-                    } else {
-#pragma unroll
-                        for (int p = 0; p < NP1; ++p) x[p] = xp[p];
-                    }
+                    sep_load_pattern<NP1>(sd, xr, q, tid, x);
                     sep_i32* yq = yr + SEP_NW1 * q;
                     sep_windows<NP1>(x, SEP_M1, SEP_NW1, SEP_D1, sd.d1_mul, sd.d1_sh,
                                      [&](int k, sep_i32 v) { yq[k] = v; });
@@ -232,12 +248,138 @@ __device__ __forceinline__ void sep_chain_body(const SepDev& sd, const sep_i32* 
     }
 }
 
+
+#if defined(SEP_JIT) && defined(SEP_REG)
+// Register-resident column filter (JIT only: it needs p2, L2 and the window masks as literals).  Thread t owns f1's
+// repetitions q = t + 256 i (i < SEP_RPT) and so the Y columns nw1 q .. nw1 q + nw1 - 1 that f2 reads (f2 filters
+// each column on its own): the f2 window sums accumulate in registers as the Y rows are produced -- the hand-WLF
+// of the specialised K-5 kernel, here for any separable pair of run-time filters.  A Y row belongs to at most
+// kRegNB = ceil(L2 / p2) bands; with the row loop unrolled over kRegNB p2 rows, a row's offset in each band and
+// the band's accumulator slot are compile-time constants (the slot of band b is b mod kRegNB; a band's first row
+// initialises its slot, its row L2 - 1 emits it).  One CTA barrier per row (the staged X row), no Y ring.
+constexpr int kRegNB = (SEP_L2 + SEP_P2 - 1) / SEP_P2;
+#ifndef SEP_NBUF
+#define SEP_NBUF kSepNB
+#endif
+constexpr int kRegBuf = SEP_NBUF;   // X row buffers (kRegBuf - 1 rows in flight per CTA)
+constexpr int kRegPeriod = kRegNB * SEP_P2;
+
+template <int NP1>
+__device__ __forceinline__ void sep_reg_body(const SepDev& sd, const sep_i32* __restrict__ X, sep_i32* __restrict__ Z,
+                                             sep_i32* sm) {
+    sep_i32* xb = sm;   // [kRegBuf][xstride]
+    const int tid = threadIdx.x;
+    for (sep_i32 unit = blockIdx.x; unit < sd.nunits; unit += gridDim.x) {
+        const sep_i32 plane = unit / sd.runs, run = unit - plane * sd.runs;
+        const sep_i32 b0 = run * sd.nb, b1 = min(b0 + sd.nb, sd.R2);
+        const sep_i32 nrows = (b1 - b0 - 1) * SEP_P2 + SEP_L2;
+        const sep_i32* Xp = X + sep_i64(plane) * SEP_HX * SEP_WX;
+        sep_i32* Zp = Z + sep_i64(plane) * SEP_HZ * SEP_WY;
+        sep_i32 xrow_next = sep_i32((sep_i64(sd.o2r) + sep_i64(SEP_P2) * b0) % SEP_HY) + sd.o1r;
+        if (xrow_next >= SEP_HX) xrow_next -= SEP_HX;
+        sep_i32 staged = 0;
+        auto issue = [&]() {
+            if (staged < nrows) {
+                sep_stage_row(sd, Xp + sep_i64(xrow_next) * SEP_WX, sep_smem_u32(xb + (staged % kRegBuf) * SEP_XSTRIDE),
+                              tid);
+                ++staged;
+                if (++xrow_next == SEP_HX) xrow_next = 0;
+            }
+            sep_cp_commit();
+        };
+#pragma unroll
+        for (int i = 0; i < kRegBuf - 1; ++i) issue();
+        sep_i32 acc[kRegNB][SEP_NW2][SEP_RPT][SEP_NW1];
+#pragma unroll
+        for (int b = 0; b < kRegNB; ++b)
+#pragma unroll
+            for (int k2 = 0; k2 < SEP_NW2; ++k2)
+#pragma unroll
+                for (int i = 0; i < SEP_RPT; ++i)
+#pragma unroll
+                    for (int c = 0; c < SEP_NW1; ++c) acc[b][k2][i][c] = 0;
+        for (sep_i32 j0 = 0; j0 < nrows; j0 += kRegPeriod) {
+#pragma unroll
+            for (int u = 0; u < kRegPeriod; ++u) {
+                const sep_i32 j = j0 + u;
+                if (j >= nrows) break;
+                sep_cp_wait<kRegBuf - 2>();
+                // row j staged by every thread, and every thread is done with row j - 1: only now may its buffer
+                // take row j + kRegBuf - 1 (this kernel has no second barrier per row to order that)
+                __syncthreads();
+                issue();
+                const sep_i32* xr = xb + (j % kRegBuf) * SEP_XSTRIDE;
+                sep_i32 y[SEP_RPT][SEP_NW1];
+#pragma unroll
+                for (int i = 0; i < SEP_RPT; ++i) {
+                    // (threads past the last repetition compute a copy of it and store nothing)
+                    const sep_i32 q = min(tid + kSepThreads * i, SEP_R1 - 1);
+                    sep_i32 x[NP1];
+                    sep_load_pattern<NP1>(sd, xr, q, tid, x);
+#pragma unroll
+                    for (int k = 0; k < SEP_NW1; ++k) {
+                        sep_i32 S = 0;
+#pragma unroll
+                        for (int p = 0; p < NP1; ++p)
+                            if (sep_m1{}(k, p)) S += x[p];
+                        y[i][k] = SEP_TASK(S, SEP_D1, 0u, 0u);
+                    }
+                }
+                // the row's offset in the band starting d band steps earlier: u % p2 + d p2 (all literals)
+#pragma unroll
+                for (int d = 0; d < kRegNB; ++d) {
+                    const int t = u % SEP_P2 + d * SEP_P2;
+                    const int slot = ((u / SEP_P2 - d) % kRegNB + kRegNB) % kRegNB;
+                    if (t < SEP_L2) {
+#pragma unroll
+                        for (int k2 = 0; k2 < SEP_NW2; ++k2) {
+                            const bool in = sep_m2{}(k2, t);
+#pragma unroll
+                            for (int i = 0; i < SEP_RPT; ++i)
+#pragma unroll
+                                for (int c = 0; c < SEP_NW1; ++c) {
+                                    if (t == 0)
+                                        acc[slot][k2][i][c] = in ? y[i][c] : 0;
+                                    else if (in)
+                                        acc[slot][k2][i][c] += y[i][c];
+                                }
+                        }
+                    }
+                    if (t == SEP_L2 - 1 && j >= SEP_L2 - 1) {   // band (j - L2 + 1) / p2 of the unit is complete
+                        const sep_i32 band = b0 + (j - (SEP_L2 - 1)) / SEP_P2;
+                        sep_i32* zb = Zp + sep_i64(SEP_NW2) * band * SEP_WY;
+#pragma unroll
+                        for (int i = 0; i < SEP_RPT; ++i) {
+                            const sep_i32 q = tid + kSepThreads * i;
+                            if (q < SEP_R1) {
+#pragma unroll
+                                for (int k2 = 0; k2 < SEP_NW2; ++k2)
+#pragma unroll
+                                    for (int c = 0; c < SEP_NW1; ++c)
+                                        zb[sep_i64(k2) * SEP_WY + SEP_NW1 * q + c] =
+                                            SEP_TASK(acc[slot][k2][i][c], SEP_D2, 0u, 0u);
+                            }
+                        }
+                    }
+                }
+            }
+        }
+        sep_cp_wait<0>();
+        __syncthreads();   // the next unit restages the buffers
+    }
+}
+#endif
+
 #ifdef SEP_JIT
 extern "C" __global__ void __launch_bounds__(kSepThreads) sep_chain_jit(const __grid_constant__ SepDev sd,
                                                                         const sep_i32* __restrict__ X,
                                                                         sep_i32* __restrict__ Z) {
     extern __shared__ __align__(16) sep_i32 sep_sm[];
+#ifdef SEP_REG
+    sep_reg_body<SEP_NP1>(sd, X, Z, sep_sm);
+#else
     sep_chain_body<SEP_NP1, SEP_NP2>(sd, X, Z, sep_sm);
+#endif
 }
 #endif
 

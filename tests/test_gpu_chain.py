@@ -22,8 +22,10 @@ def _task_c(G, starts, L, d):
 
 
 @pytest.mark.parametrize("shape", [(2, 1080, 1920), (3, 288, 352), (2, 27, 720), (1, 9, 64), (2, 36, 1000),
-                                   (1, 2160, 3840)])
+                                   (1, 2160, 3840), (240, 1080, 1920)])
 def test_chain_h_then_v_equals_fused_downscaler(orc, shape):
+    """(240 HD planes: every SM busy with several CTAs for a while -- the staging ring's buffer reuse under load;
+    a missing barrier between a row's reads and its buffer's next copy showed up only at this scale.)"""
     P, H, W = shape
     xh = synth.frames(51, 0, 1, P, H, W, "uniform")[0]
     x = torch.from_numpy(xh).cuda()
@@ -34,7 +36,7 @@ def test_chain_h_then_v_equals_fused_downscaler(orc, shape):
     assert aol.last_kernel() == "sep_chain_jit"
     zf, _ = aol.downscale_frame(x.unsqueeze(1))
     assert torch.equal(z, zf[:, 0])
-    if H * W <= 1080 * 1920:
+    if P * H * W <= 3 * 1080 * 1920:
         assert np.array_equal(z.cpu().numpy(), orc.downscale_v(orc.downscale_h(xh)))
 
 
