@@ -238,7 +238,7 @@ def test_fused_u8_two_reps_per_thread(orc, W):
 
 @pytest.mark.parametrize("shape,kernel", [
     ((1, 3, 1080, 1920), 1), ((2, 3, 288, 352), 1), ((2, 3, 36, 1040), 1), ((2, 3, 36, 128), 1),
-    ((1, 2, 18, 40), 2), ((2, 3, 36, 128), 2),
+    ((1, 2, 18, 40), 2), ((2, 3, 36, 128), 2), ((1, 3, 2160, 3840), 1), ((2, 1, 54, 4096), 1), ((3, 3, 90, 1920), 1),
 ])
 def test_fused_u8_int16_output(orc, shape, kernel):
     """NEXT row f1's int16 output option: 8-bit samples give outputs in [-5, 255]; stored as int16 they are
@@ -254,6 +254,9 @@ def test_fused_u8_int16_output(orc, shape, kernel):
     z, cs = aol.downscale_frame(x8, checksums=True, opts=opts, out_dtype=torch.int16)
     z2, _ = aol.downscale_frame(x8, opts=opts, out_dtype=torch.int16)
     torch.cuda.synchronize()
+    if kernel == 1 and W in (1920, 3840, 4096):
+        # the halo-last multi-CTA instantiations: 4 CTAs/SM of 160 threads (HD), 2 of 288 (4K, 4096)
+        assert plan["ctas_per_sm"] == (4 if W == 1920 else 2), plan
     assert z.dtype == torch.int16
     assert np.array_equal(z.cpu().numpy().astype(np.int32), zo)
     assert np.array_equal(z2.cpu().numpy().astype(np.int32), zo)
