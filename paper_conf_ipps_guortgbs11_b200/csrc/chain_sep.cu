@@ -237,7 +237,7 @@ const Nvrtc& nvrtc() {
 }
 
 // f1 repetitions per thread of the register-resident column filter (sep_reg_body), 0 when it does not apply: at
-// most two repetitions per thread and 64 accumulators (AOL_SEP_REG=0 keeps the Y ring, for A/B measurements).
+// most four repetitions per thread and 64 accumulators (AOL_SEP_REG=0 keeps the Y ring, for A/B measurements).
 int sep_reg_rpt(const SepDev& sd) {
     static const bool enabled = [] {
         const char* e = std::getenv("AOL_SEP_REG");
@@ -245,7 +245,7 @@ int sep_reg_rpt(const SepDev& sd) {
     }();
     const int rpt = (sd.R1 + kSepThreads - 1) / kSepThreads;
     const int nbl = (sd.L2 + sd.p2 - 1) / sd.p2;
-    return enabled && rpt <= 2 && nbl * sd.nw2 * sd.nw1 * rpt <= 64 ? rpt : 0;
+    return enabled && rpt <= 4 && nbl * sd.nw2 * sd.nw1 * rpt <= 64 ? rpt : 0;
 }
 
 // X row buffers of the register-resident kernel (AOL_SEP_NBUF overrides, for A/B measurements)
@@ -395,6 +395,43 @@ bool launch_sep_chain(const aol_filter_t* f1, const aol_filter_t* f2, const int3
         *st = AOL_E_CUDA;
     }
     return true;
+}
+
+// A single filter of the chain's shape runs as a chain with an identity partner (one pattern element, one window of
+// length 1, divisor 1: T(S) = S/1 - S%1 = S): a row filter f as f -> identity column filter on its output, a
+// column filter as identity row filter on its input -> f.  Only when the run-time specialised kernel is available:
+// the statically compiled chain kernel is no faster than aol_filter_apply's own kernel for one repetition.
+bool launch_sep_single(const aol_filter_t* f, const int32_t* d_in, int32_t* d_out, cudaStream_t s, aol_status_t* st) {
+    if (!sep_jit_enabled() || !nvrtc().ok) return false;
+    const int n = f->in.array_rank;
+    if (n < 2 || f->in.pattern_rank != 1) return false;
+    const int row = n - 2, col = n - 1;
+    aol_filter_t id;
+    std::memset(&id, 0, sizeof id);
+    id.n_windows = 1;
+    id.window_len = 1;
+    id.divisor = 1;
+    auto ident = [&](aol_tiler_t& t, const int64_t* shape, int fit_dim) {
+        t.array_rank = t.rep_rank = n;
+        t.pattern_rank = 1;
+        t.pattern_shape[0] = 1;
+        for (int a = 0; a < n; ++a) {
+            t.array_shape[a] = t.rep_shape[a] = shape[a];
+            t.paving[a][a] = 1;
+            t.fitting[a][0] = a == fit_dim ? 1 : 0;
+        }
+    };
+    if (f->in.fitting[col][0] == 1) {   // a row filter, then the identity down the columns of its output
+        ident(id.in, f->out.array_shape, row);
+        ident(id.out, f->out.array_shape, row);
+        return launch_sep_chain(f, &id, d_in, d_out, s, st);
+    }
+    if (f->in.fitting[row][0] == 1) {   // the identity along the rows of its input, then a column filter
+        ident(id.in, f->in.array_shape, col);
+        ident(id.out, f->in.array_shape, col);
+        return launch_sep_chain(&id, f, d_in, d_out, s, st);
+    }
+    return false;
 }
 
 void set_sep_jit(int on) { g_sep_jit.store(on ? 1 : 0); }

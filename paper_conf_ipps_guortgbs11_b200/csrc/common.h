@@ -89,6 +89,9 @@ aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t i
 // case (nothing done); true: handled, *st = the outcome.
 bool launch_sep_chain(const aol_filter_t* f1, const aol_filter_t* f2, const int32_t* d_in, int32_t* d_out,
                       cudaStream_t s, aol_status_t* st);
+// aol_filter_apply for a single row filter or column filter: the separable chain kernel with an identity partner
+// filter, specialised at run time (false when NVRTC is absent or the filter is not of that shape).
+bool launch_sep_single(const aol_filter_t* f, const int32_t* d_in, int32_t* d_out, cudaStream_t s, aol_status_t* st);
 
 aol_status_t launch_downscale_h(const int32_t* d_in, int32_t* d_out, int64_t planes, int64_t H, int64_t W,
                                 cudaStream_t s);

@@ -547,6 +547,9 @@ aol_status_t aol_filter_apply(const aol_filter_t* f, const int32_t* d_in, int32_
     if (!d_in || !d_out) return fail(AOL_E_INVALID, "null buffer");
     if ((reinterpret_cast<uintptr_t>(d_in) | reinterpret_cast<uintptr_t>(d_out)) % 4)
         return fail(AOL_E_ALIGN, "buffers must be 4-byte aligned");
+    // a row filter or a column filter (the paper's H and V, any run-time parameters): the separable chain kernel
+    // specialised at run time, with an identity partner
+    if (launch_sep_single(f, d_in, d_out, s, &st)) return st;
     FilterDev fd;
     std::memset(&fd, 0, sizeof fd);
     fd.ra_in = f->in.array_rank;

@@ -199,3 +199,48 @@ def test_unfusable_chain_needs_a_workspace(orc):
     torch.cuda.synchronize()
     y = aol.filter_apply(fh2, x)
     assert torch.equal(z, aol.filter_apply(fv, y))
+
+
+@pytest.mark.parametrize("seed", range(24))
+def test_random_single_row_and_column_filters(orc, seed):
+    """aol_filter_apply on ONE row filter or ONE column filter with random parameters (lead dims, pattern lengths,
+    paving steps, wrapping origins, windows, divisors of either sign): these run the separable chain kernel,
+    specialised at run time, with an identity partner filter.  Expected: the oracle's gather -> C task -> scatter."""
+    rng = np.random.default_rng(9100 + seed)
+    n = int(rng.integers(2, 5))
+    lead = [int(rng.integers(1, 4)) for _ in range(n - 2)]
+    H, W = int(rng.integers(1, 40)), int(rng.integers(4, 1200))
+    if seed % 3 == 0:
+        W = 4 * int(rng.integers(1, 300))
+    L = int(rng.integers(1, 17))
+    ln = int(rng.integers(1, L + 1))
+    nw = int(rng.integers(1, 9))
+    st = [int(rng.integers(0, L - ln + 1)) for _ in range(nw)]
+    d = int(rng.choice([1, 2, 3, 6, 7, -1, -6, 100]))
+    ones = [1] * (n - 2)
+    e_col = [[0]] * (n - 1) + [[1]]
+    e_row = [[0]] * (n - 2) + [[1], [0]]
+    row_filter = seed % 2 == 0
+    if row_filter:
+        p = int(rng.integers(1, 12))
+        R = int(rng.integers(1, max(2, 2 * W // p)))
+        o = [0] * (n - 2) + [int(rng.integers(-2 * H, 2 * H + 1)), int(rng.integers(-2 * W, 2 * W + 1))]
+        ax, ay = lead + [H, W], lead + [H, nw * R]
+        ti = (ax, lead + [H, R], [L], o, _eye(n, ones + [1, p]), e_col)
+        to = (ay, lead + [H, R], [nw], [0] * n, _eye(n, ones + [1, nw]), e_col)
+    else:
+        p = int(rng.integers(1, L + 1))
+        R = int(rng.integers(1, 12))
+        o = [0] * (n - 2) + [int(rng.integers(-2 * H, 2 * H + 1)), 0]
+        ax, ay = lead + [H, W], lead + [nw * R, W]
+        ti = (ax, lead + [R, W], [L], o, _eye(n, ones + [p, 1]), e_row)
+        to = (ay, lead + [R, W], [nw], [0] * n, _eye(n, ones + [nw, 1]), e_row)
+    xh = np.asarray(rng.integers(-3000, 3000, size=ax)).astype(np.int32)
+    bg = np.full(ay, -7, np.int32)
+    want = orc.scatter(orc.make_tiler(*to), _task_c(orc.gather(orc.make_tiler(*ti), xh), st, ln, d), bg)
+    f = aol.make_filter(aol.make_tiler(*ti), aol.make_tiler(*to), st, ln, d)
+    out = torch.from_numpy(bg.copy()).cuda()
+    aol.filter_apply(f, torch.from_numpy(xh).cuda(), out=out)
+    torch.cuda.synchronize()
+    assert aol.last_kernel() == "sep_chain_jit"
+    assert np.array_equal(out.cpu().numpy(), want)
