@@ -43,6 +43,12 @@ AOL_API const char* aol_debug_last_kernel(void);
  * the default unless AOL_CHAIN_JIT=0) or the statically compiled generic one (off).  Same results. */
 AOL_API void aol_debug_set_chain_jit(int on);
 
+/* Test hook, no GPU needed: compile (with NVRTC, without loading) the run-time specialised separable chain kernel
+ * aol_filter_chain_apply would build for f1 -> f2.  Returns 1 (compiled; log = "register-resident" or "ring", the
+ * kernel body chosen), 0 (not a separable chain; log = why), -1 (NVRTC not available), -2 (compilation failed;
+ * log = the NVRTC log).  log may be NULL. */
+AOL_API int aol_debug_sep_jit_compile(const aol_filter_t* f1, const aol_filter_t* f2, char* log, size_t cap);
+
 #ifdef __cplusplus
 }
 #endif

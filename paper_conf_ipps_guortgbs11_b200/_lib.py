@@ -115,6 +115,7 @@ SIGNATURES = {
     "aol_debug_fail_next_launches": ([ctypes.c_int], None),
     "aol_debug_last_kernel": ([], ctypes.c_char_p),
     "aol_debug_set_chain_jit": ([ctypes.c_int], None),
+    "aol_debug_sep_jit_compile": ([_FP, _FP, ctypes.c_char_p, ctypes.c_size_t], ctypes.c_int),
     "aol_frame_plan_create": ([_P, ctypes.c_int, _P, ctypes.c_int, _I64, _I64, _I64, _I64,
                                ctypes.POINTER(aol_launch_opts_t), ctypes.POINTER(_P)], _ST),
     "aol_frame_plan_launch": ([_P, _P, _P], _ST),

@@ -248,14 +248,25 @@ int sep_reg_rpt(const SepDev& sd) {
     return enabled && rpt <= 4 && nbl * sd.nw2 * sd.nw1 * rpt <= 64 ? rpt : 0;
 }
 
-// X row buffers of the register-resident kernel (AOL_SEP_NBUF overrides, for A/B measurements)
-int sep_reg_nbuf() {
-    static const int n = [] {
+// Row staging of the register-resident kernel: 1-D bulk copies (TMA) when the rows are 16-byte aligned (sd.vec),
+// else cp.async chunks; AOL_SEP_BULK=0 forces cp.async (A/B measurements).
+bool sep_bulk(const SepDev& sd) {
+    static const bool no_bulk = [] {
+        const char* e = std::getenv("AOL_SEP_BULK");
+        return e && e[0] == '0';
+    }();
+    return sd.vec && !no_bulk;
+}
+
+// X row buffers of the register-resident kernel: 4 with bulk copies (1.282 ms vs 1.330 at 3 and 1.370 at 6), 3 with
+// cp.async (1.358 vs 1.364 at 4, 1.51 at 5-6; profiles/r02_f3_reg_sweep.jsonl).  AOL_SEP_NBUF overrides (A/B).
+int sep_reg_nbuf(const SepDev& sd) {
+    static const int forced = [] {
         const char* e = std::getenv("AOL_SEP_NBUF");
         const int v = e ? std::atoi(e) : 0;
-        return v >= 2 && v <= 16 ? v : 3;   // 3: 1.358 ms vs 1.364 at 4, 1.51 at 5-6 (profiles/r02_f3_reg_sweep.jsonl)
+        return v >= 2 && v <= 16 ? v : 0;
     }();
-    return n;
+    return forced ? forced : sep_bulk(sd) ? 4 : 3;
 }
 
 // The literal parameters the specialised kernel is compiled for (also its cache key): the filters' patterns,
@@ -275,7 +286,18 @@ std::string sep_preamble(const aol_filter_t* f1, const aol_filter_t* f2, const S
                   sd.HX, sd.WX, sd.HY, sd.WY, sd.HZ, sd.R1, sd.J, sd.xstride, sd.vec, sd.o1c);
     s += b;
     if (const int rpt = sep_reg_rpt(sd)) {
-        std::snprintf(b, sizeof b, "#define SEP_REG 1\n#define SEP_RPT %d\n#define SEP_NBUF %d\n", rpt, sep_reg_nbuf());
+        std::snprintf(b, sizeof b, "#define SEP_REG 1\n#define SEP_RPT %d\n#define SEP_NBUF %d\n", rpt, sep_reg_nbuf(sd));
+        s += b;
+        if (!sep_bulk(sd)) s += "#define SEP_NO_BULK 1\n";
+        // bytes one staged row's bulk copies deliver (the last contiguous segment rounded up to 16 bytes)
+        int64_t col = sd.o1c, left = sd.J, total = 0;
+        while (left > 0) {
+            const int64_t len = std::min<int64_t>(left, sd.WX - col);
+            total += (len + 3) / 4 * 16;
+            left -= len;
+            col = 0;
+        }
+        std::snprintf(b, sizeof b, "#define SEP_BULK_BYTES %lldu\n", static_cast<long long>(total));
         s += b;
     }
     for (int f = 0; f < 2; ++f) {
@@ -304,6 +326,37 @@ bool sep_jit_enabled() {
     return v != 0;
 }
 
+// NVRTC: the kernel body with the preamble's literals -> a cubin for sm_100a (false, the log in *note, on failure).
+bool sep_nvrtc_compile(const std::string& pre, std::vector<char>* cubin, std::string* note) {
+    const Nvrtc& nv = nvrtc();
+    if (!nv.ok) {
+        *note = "NVRTC not available";
+        return false;
+    }
+    const std::string src = pre + kSepBodySrc;
+    void* prog = nullptr;
+    if (nv.create(&prog, src.c_str(), "aol_sep_chain.cu", 0, nullptr, nullptr) != 0) {
+        *note = "nvrtcCreateProgram failed";
+        return false;
+    }
+    const char* opts[] = {"--gpu-architecture=sm_100a", "-std=c++17", "-lineinfo"};
+    bool ok = nv.compile(prog, 3, opts) == 0;
+    if (ok) {
+        size_t n = 0;
+        nv.cubin_size(prog, &n);
+        cubin->resize(n);
+        nv.cubin(prog, cubin->data());
+    } else {
+        size_t n = 0;
+        nv.log_size(prog, &n);
+        std::string log(n, '\0');
+        nv.log(prog, &log[0]);
+        *note = "NVRTC: " + log;
+    }
+    nv.destroy(&prog);
+    return ok;
+}
+
 // The specialised kernel for these filters: compiled on first use, then cached (per process; a library loaded
 // through the runtime is available on every device).  nullptr: NVRTC missing or the compilation failed (the
 // reason is kept for aol_last_error-free diagnostics in jit_note).
@@ -320,32 +373,17 @@ const void* sep_jit_kernel(const aol_filter_t* f1, const aol_filter_t* f2, const
     auto it = g_jit_cache.find(pre);
     if (it != g_jit_cache.end()) return it->second;
     const void* kern = nullptr;
-    const std::string src = pre + kSepBodySrc;
-    void* prog = nullptr;
-    if (nv.create(&prog, src.c_str(), "aol_sep_chain.cu", 0, nullptr, nullptr) == 0) {
-        const char* opts[] = {"--gpu-architecture=sm_100a", "-std=c++17", "-lineinfo"};
-        if (nv.compile(prog, 3, opts) == 0) {
-            size_t n = 0;
-            nv.cubin_size(prog, &n);
-            std::vector<char> cubin(n);
-            nv.cubin(prog, cubin.data());
-            cudaLibrary_t lib = nullptr;
-            cudaKernel_t k = nullptr;
-            cudaError_t le = cudaLibraryLoadData(&lib, cubin.data(), nullptr, nullptr, 0, nullptr, nullptr, 0);
-            if (le == cudaSuccess) le = cudaLibraryGetKernel(&k, lib, "sep_chain_jit");
-            if (le == cudaSuccess)
-                kern = reinterpret_cast<const void*>(k);   // the library stays loaded for the process
-            else
-                g_jit_note = std::string("loading the compiled kernel failed: ") + cudaGetErrorString(le);
-            cudaGetLastError();
-        } else {
-            size_t n = 0;
-            nv.log_size(prog, &n);
-            std::string log(n, '\0');
-            nv.log(prog, &log[0]);
-            g_jit_note = "NVRTC: " + log;
-        }
-        nv.destroy(&prog);
+    std::vector<char> cubin;
+    if (sep_nvrtc_compile(pre, &cubin, &g_jit_note)) {
+        cudaLibrary_t lib = nullptr;
+        cudaKernel_t k = nullptr;
+        cudaError_t le = cudaLibraryLoadData(&lib, cubin.data(), nullptr, nullptr, 0, nullptr, nullptr, 0);
+        if (le == cudaSuccess) le = cudaLibraryGetKernel(&k, lib, "sep_chain_jit");
+        if (le == cudaSuccess)
+            kern = reinterpret_cast<const void*>(k);   // the library stays loaded for the process
+        else
+            g_jit_note = std::string("loading the compiled kernel failed: ") + cudaGetErrorString(le);
+        cudaGetLastError();
     }
     if (!kern && std::getenv("AOL_JIT_VERBOSE")) std::fprintf(stderr, "aol: chain JIT failed: %s\n", g_jit_note.c_str());
     g_jit_cache.emplace(pre, kern);   // failures are cached too: the static kernel serves those filters
@@ -378,7 +416,7 @@ bool launch_sep_chain(const aol_filter_t* f1, const aol_filter_t* f2, const int3
     const void* kern = jit ? jit : reinterpret_cast<const void*>(sep_kernel_for(sd.L1, sd.L2));
     const char* name = jit ? "sep_chain_jit" : "sep_chain_kernel";
     if (jit && sep_reg_rpt(sd)) {
-        smem = int(4 * int64_t(sep_reg_nbuf()) * sd.xstride);   // no Y ring
+        smem = int((4 * int64_t(sd.xstride) + 8) * sep_reg_nbuf(sd));   // row buffers + their mbarriers, no Y ring
         sep_set_bands(&sd, 24, dev);   // longer units: 1.358 ms at 24 bands vs 1.386 at 16 and 1.440 at 8
     }
     *st = kernel_smem(kern, smem);
@@ -436,6 +474,35 @@ bool launch_sep_single(const aol_filter_t* f, const int32_t* d_in, int32_t* d_ou
 
 void set_sep_jit(int on) { g_sep_jit.store(on ? 1 : 0); }
 
+// CPU-testable: compile (not load) the run-time specialised kernel for a separable filter pair.
+int sep_jit_compile_check(const aol_filter_t* f1, const aol_filter_t* f2, char* log, size_t cap) {
+    DeviceInfo dev;
+    if (device_info(&dev) != AOL_OK) dev = DeviceInfo{0, 148, 232448, 233472};   // no GPU: B200's figures
+    cudaGetLastError();
+    SepDev sd;
+    int smem = 0;
+    const char* why = "";
+    if (!plan_sep(f1, f2, dev, &sd, &smem, &why)) {
+        if (log && cap) std::snprintf(log, cap, "%s", why);
+        return 0;
+    }
+    if (!nvrtc().ok) {
+        if (log && cap) std::snprintf(log, cap, "NVRTC not available");
+        return -1;
+    }
+    std::vector<char> cubin;
+    std::string note;
+    const bool ok = sep_nvrtc_compile(sep_preamble(f1, f2, sd), &cubin, &note);
+    if (log && cap) std::snprintf(log, cap, "%s", ok ? (sep_reg_rpt(sd) ? "register-resident" : "ring") : note.c_str());
+    return ok ? 1 : -2;
+}
+
 }  // namespace aol
 
 extern "C" AOL_API void aol_debug_set_chain_jit(int on) { aol::set_sep_jit(on); }
+
+extern "C" AOL_API int aol_debug_sep_jit_compile(const aol_filter_t* f1, const aol_filter_t* f2, char* log,
+                                                 size_t cap) {
+    if (!f1 || !f2) return 0;
+    return aol::sep_jit_compile_check(f1, f2, log, cap);
+}

@@ -264,11 +264,60 @@ constexpr int kRegNB = (SEP_L2 + SEP_P2 - 1) / SEP_P2;
 constexpr int kRegBuf = SEP_NBUF;   // X row buffers (kRegBuf - 1 rows in flight per CTA)
 constexpr int kRegPeriod = kRegNB * SEP_P2;
 
+#if SEP_VEC && !defined(SEP_NO_BULK) && defined(SEP_BULK_BYTES)
+// TMA staging (16-byte-aligned rows): thread 0 copies a whole X row with 1-D bulk copies -- one per contiguous
+// segment of the J elements from column o1c (mod WX), the last one rounded up to 16 bytes (within the row: WX and o1c
+// are multiples of 4; the overhang lands in the buffer's slack) -- completing on the buffer's mbarrier, instead of
+// every thread issuing 16-byte cp.async chunks: fewer, larger requests (HBM efficiency).
+#define SEP_BULK 1
+constexpr sep_u32 kSepBulkBytes = SEP_BULK_BYTES;   // bytes one row's copies deliver (host-computed expect-tx count)
+__device__ __forceinline__ void sep_mbar_init(sep_u32 bar) {
+    asm volatile("mbarrier.init.shared::cta.b64 [%0], 1;" ::"r"(bar) : "memory");
+}
+__device__ __forceinline__ void sep_bulk_row(const sep_i32* src_row, sep_u32 dst, sep_u32 bar) {
+    asm volatile("{\n\t.reg .b64 st;\n\tmbarrier.arrive.expect_tx.shared::cta.b64 st, [%0], %1;\n\t}" ::"r"(bar),
+                 "r"(kSepBulkBytes)
+                 : "memory");
+    sep_i32 col = SEP_O1C, left = SEP_J, off = 0;
+#pragma unroll 1
+    while (left > 0) {
+        const sep_i32 len = left < SEP_WX - col ? left : SEP_WX - col;
+        asm volatile("cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];" ::"r"(
+                         dst + 4u * sep_u32(off)),
+                     "l"(src_row + col), "r"(sep_u32((len + 3) / 4) * 16u), "r"(bar)
+                     : "memory");
+        off += len;
+        left -= len;
+        col = 0;
+    }
+}
+__device__ __forceinline__ void sep_mbar_wait(sep_u32 bar, sep_u32 parity) {
+    sep_u32 ok;
+    do {
+        asm volatile("{\n\t.reg .pred p;\n\tmbarrier.try_wait.parity.shared::cta.b64 p, [%1], %2;\n\t"
+                     "selp.u32 %0, 1, 0, p;\n\t}"
+                     : "=r"(ok)
+                     : "r"(bar), "r"(parity)
+                     : "memory");
+    } while (!ok);
+}
+#endif
+
 template <int NP1>
 __device__ __forceinline__ void sep_reg_body(const SepDev& sd, const sep_i32* __restrict__ X, sep_i32* __restrict__ Z,
                                              sep_i32* sm) {
     sep_i32* xb = sm;   // [kRegBuf][xstride]
     const int tid = threadIdx.x;
+#ifdef SEP_BULK
+    // one mbarrier per row buffer after the buffers; a buffer's k-th use completes phase k
+    const sep_u32 bars = sep_smem_u32(sm + kRegBuf * SEP_XSTRIDE);
+    if (tid == 0) {
+        for (int b = 0; b < kRegBuf; ++b) sep_mbar_init(bars + 8u * sep_u32(b));
+        asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+    }
+    __syncthreads();
+    sep_u32 issued = 0, consumed = 0;   // rows staged / consumed by this CTA over all its units
+#endif
     for (sep_i32 unit = blockIdx.x; unit < sd.nunits; unit += gridDim.x) {
         const sep_i32 plane = unit / sd.runs, run = unit - plane * sd.runs;
         const sep_i32 b0 = run * sd.nb, b1 = min(b0 + sd.nb, sd.R2);
@@ -280,12 +329,21 @@ __device__ __forceinline__ void sep_reg_body(const SepDev& sd, const sep_i32* __
         sep_i32 staged = 0;
         auto issue = [&]() {
             if (staged < nrows) {
+#ifdef SEP_BULK
+                const sep_u32 b = issued % kRegBuf;
+                if (tid == 0)
+                    sep_bulk_row(Xp + sep_i64(xrow_next) * SEP_WX, sep_smem_u32(xb + b * SEP_XSTRIDE), bars + 8u * b);
+                ++issued;
+#else
                 sep_stage_row(sd, Xp + sep_i64(xrow_next) * SEP_WX, sep_smem_u32(xb + (staged % kRegBuf) * SEP_XSTRIDE),
                               tid);
+#endif
                 ++staged;
                 if (++xrow_next == SEP_HX) xrow_next = 0;
             }
+#ifndef SEP_BULK
             sep_cp_commit();
+#endif
         };
 #pragma unroll
         for (int i = 0; i < kRegBuf - 1; ++i) issue();
@@ -303,12 +361,19 @@ __device__ __forceinline__ void sep_reg_body(const SepDev& sd, const sep_i32* __
             for (int u = 0; u < kRegPeriod; ++u) {
                 const sep_i32 j = j0 + u;
                 if (j >= nrows) break;
+#ifdef SEP_BULK
+                const sep_u32 cb = consumed % kRegBuf;
+                sep_mbar_wait(bars + 8u * cb, (consumed / kRegBuf) & 1u);   // row j has landed
+                ++consumed;
+                const sep_i32* xr = xb + cb * SEP_XSTRIDE;
+#else
                 sep_cp_wait<kRegBuf - 2>();
-                // row j staged by every thread, and every thread is done with row j - 1: only now may its buffer
-                // take row j + kRegBuf - 1 (this kernel has no second barrier per row to order that)
+                const sep_i32* xr = xb + (j % kRegBuf) * SEP_XSTRIDE;
+#endif
+                // row j staged, and every thread is done with row j - 1: only now may its buffer take row
+                // j + kRegBuf - 1 (this kernel has no second barrier per row to order that)
                 __syncthreads();
                 issue();
-                const sep_i32* xr = xb + (j % kRegBuf) * SEP_XSTRIDE;
                 sep_i32 y[SEP_RPT][SEP_NW1];
 #pragma unroll
                 for (int i = 0; i < SEP_RPT; ++i) {
@@ -364,14 +429,21 @@ __device__ __forceinline__ void sep_reg_body(const SepDev& sd, const sep_i32* __
                 }
             }
         }
+#ifndef SEP_BULK
         sep_cp_wait<0>();
+#endif
         __syncthreads();   // the next unit restages the buffers
     }
 }
 #endif
 
 #ifdef SEP_JIT
-extern "C" __global__ void __launch_bounds__(kSepThreads) sep_chain_jit(const __grid_constant__ SepDev sd,
+#ifdef SEP_REG
+#define SEP_MIN_BLOCKS 4   // 64 registers: 4 CTAs of 256 threads per SM
+#else
+#define SEP_MIN_BLOCKS 1
+#endif
+extern "C" __global__ void __launch_bounds__(kSepThreads, SEP_MIN_BLOCKS) sep_chain_jit(const __grid_constant__ SepDev sd,
                                                                         const sep_i32* __restrict__ X,
                                                                         sep_i32* __restrict__ Z) {
     extern __shared__ __align__(16) sep_i32 sep_sm[];
