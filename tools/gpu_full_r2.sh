@@ -7,7 +7,7 @@ T=${TAG:-r02_full}
 nvidia-smi --query-gpu=name,clocks.sm,clocks.max.sm,power.draw --format=csv > gpurun_out/${T}_gpu.txt 2>&1
 timeout 1500 python -m pytest tests -m gpu -q > gpurun_out/${T}_pytest_gpu.log 2>&1; echo "pytest rc=$?" >> gpurun_out/${T}_pytest_gpu.log
 timeout 300 python -c "import __graft_entry__ as g; g.smoke()" > gpurun_out/${T}_smoke.log 2>&1; echo "smoke rc=$?" >> gpurun_out/${T}_smoke.log
-timeout 900 python bench.py > gpurun_out/${T}_bench.json 2> gpurun_out/${T}_bench.err
+s0=$(date +%s); timeout 900 python bench.py > gpurun_out/${T}_bench.json 2> gpurun_out/${T}_bench.err; echo "default bench wall s: $(( $(date +%s) - s0 ))" > gpurun_out/${T}_bench_wall.txt
 timeout 600 python bench.py --dtype u8 --no-cpu-baseline > gpurun_out/${T}_bench_u8.json 2>> gpurun_out/${T}_bench.err
 timeout 600 python bench.py --dtype u8 --out-dtype i16 --no-cpu-baseline > gpurun_out/${T}_bench_u8i16.json 2>> gpurun_out/${T}_bench.err
 timeout 600 python bench.py --dtype rgb8 --no-cpu-baseline > gpurun_out/${T}_bench_rgb8.json 2>> gpurun_out/${T}_bench.err
