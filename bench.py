@@ -666,6 +666,19 @@ def record_f3(aol, peak, a, frame0, F, d2_cs):
     y = torch.empty((P, H, 3 * (W // 8)), dtype=torch.int32, device="cuda")
     z2 = torch.empty_like(z)
     med2, _ = timed(lambda: (aol.filter_apply(fh, x, out=y), aol.filter_apply(fv, y, out=z2)), inner=2)
+    # the paper's generic-vs-specialised comparison (Section VIII-A) without run-time specialisation:
+    # the chain and the two launches on the statically compiled kernels (parameters read from the descriptors)
+    from paper_conf_ipps_guortgbs11_b200 import _lib
+    z3, z4 = torch.empty_like(z), torch.empty_like(z)
+    _lib.lib().aol_debug_set_chain_jit(0)
+    try:
+        med3, _ = timed(lambda: aol.filter_chain_apply(fh, fv, x, out=z3), inner=2, reps=5)
+        kernel3 = aol.last_kernel()
+        med4, _ = timed(lambda: (aol.filter_apply(fh, x, out=y), aol.filter_apply(fv, y, out=z4)), inner=1, reps=5)
+    finally:
+        _lib.lib().aol_debug_set_chain_jit(1)
+    static_equal = bool(torch.equal(z, z3) and torch.equal(z, z4))
+    del z3, z4
     cs = aol.frame_checksum(z.reshape(F, C, 4 * (H // 9), 3 * (W // 8)))
     torch.cuda.synchronize()
     got = cs.cpu().view(torch.int64).numpy().view(np.uint64)
@@ -677,7 +690,12 @@ def record_f3(aol, peak, a, frame0, F, d2_cs):
                       "chained in one kernel", "kernel": kernel, "ms": med, "min_ms": mn,
             "frames_per_s": F / (med / 1e3), "GBps": b / med / 1e6, "frac": b / med / 1e6 / peak,
             "two_launches_ms": med2, "two_launches_frames_per_s": F / (med2 / 1e3),
-            "two_launches_equal": two_equal, "parity": bool(np.array_equal(got, d2_cs[:F])),
+            "two_launches_equal": two_equal,
+            "static": {"kernel": kernel3, "chain_ms": med3, "two_launches_ms": med4, "equal": static_equal,
+                       "note": "the same filters without run-time specialisation (aol_debug_set_chain_jit(0)): the "
+                               "statically compiled separable chain, and each filter on the generic per-repetition "
+                               "kernel"},
+            "parity": bool(np.array_equal(got, d2_cs[:F])),
             "parity_scope": f"all {F} frame checksums equal the d2 fused kernel's (themselves vs the oracle in "
                             "cpu_baseline)",
             "timing": "CUDA events, 5 (two launches: 2) calls back to back per event pair, median of 20"}

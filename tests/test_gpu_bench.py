@@ -63,6 +63,7 @@ def test_bench_full_default_run_records_and_parity():
     assert rec["d4"]["parity"] is True and rec["d4"]["frames_per_s"] > 10000
     assert rec["wide"]["parity"] is True and rec["wide"]["kernel"] == "fused_tma_kernel"
     assert rec["f3"]["parity"] is True and rec["f3"]["two_launches_equal"] is True
+    assert rec["f3"]["static"]["equal"] is True and rec["f3"]["static"]["kernel"] == "sep_chain_kernel"
     assert len(rec["f1"]) == 4 and all(r["parity"] is True for r in rec["f1"])
     assert rec["f4"]["parity"] is True and rec["f4"]["frames_per_s"] > 100000
     assert rec["d5"]["parity"] is True and rec["d5"]["scaling"] == "strong" and rec["d5"]["n_gpus"] == 1
