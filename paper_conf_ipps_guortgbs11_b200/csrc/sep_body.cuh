@@ -121,12 +121,19 @@ __device__ __forceinline__ void sep_load_pattern(const SepDev& sd, const sep_i32
         // 16-byte aligned pattern: NP1/4 LDS.128 (scalar loads at a stride of p1 words conflict p1/gcd-way on the
         // banks).  At p1 = 8 a quarter-warp's chunks v sit in every other 16-byte bank group: lanes with bit 2 set
         // take chunks 0 and 1 in the other order, which spreads both loads over all 8 groups (conflict-free).
-        const bool swp = SEP_P1 == 8 && ((tid >> 2) & 1);
+        // (run-time specialised kernel only: with p1 read from the descriptor the swap costs the static kernel
+        // more than the conflicts it saves -- 3.65 vs 3.14 ms on the d2 workload)
+#ifdef SEP_JIT
+        constexpr bool kSwap = true;
+#else
+        constexpr bool kSwap = false;
+#endif
+        const bool swp = kSwap && SEP_P1 == 8 && ((tid >> 2) & 1);
         const int4* xp4 = reinterpret_cast<const int4*>(xp);
         int4 c[NP1 / 4 > 0 ? NP1 / 4 : 1];
 #pragma unroll
         for (int v = 0; v < NP1 / 4; ++v) c[v] = xp4[v];
-        if (NP1 >= 8) {
+        if (kSwap && NP1 >= 8) {
             const int4 L0 = xp4[swp ? 1 : 0], L1 = xp4[swp ? 0 : 1];   // load slots 0 and 1
             c[0] = swp ? L1 : L0;
             c[1] = swp ? L0 : L1;
@@ -149,8 +156,13 @@ __device__ __forceinline__ void sep_load_pattern(const SepDev& sd, const sep_i32
 // literal.)
 __device__ __forceinline__ void sep_stage_row(const SepDev& sd, const sep_i32* src, sep_u32 dst, int tid) {
     (void)sd;
-    // (one conditional subtraction when the staged span wraps at most once, o1c + J <= 2 WX)
+    // (one conditional subtraction when the staged span wraps at most once, o1c + J <= 2 WX: a literal in the
+    // run-time specialised kernel; the static one keeps the plain loop)
+#ifdef SEP_JIT
     const bool once = SEP_O1C + SEP_J <= 2 * SEP_WX;
+#else
+    constexpr bool once = false;
+#endif
     if (SEP_VEC) {   // o1c, WX multiples of 4: every 16-byte chunk lies on one side of the wrap
         for (sep_i32 c = tid; 4 * c < SEP_J; c += kSepThreads) {
             sep_i32 col = SEP_O1C + 4 * c;
