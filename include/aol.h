@@ -323,7 +323,12 @@ AOL_API aol_status_t aol_filter_preset(aol_filter_kind_t which, int64_t planes, 
 AOL_API aol_status_t aol_filter_validate(const aol_filter_t* f);
 
 /* Apply a filter: d_in int32 shaped f->in.array_shape, d_out int32 shaped f->out.array_shape
- * (cells no repetition writes keep their value).  4-byte aligned.  Async on s. */
+ * (cells no repetition writes keep their value).  4-byte aligned.  Async on s.
+ * A row filter or a column filter (pattern along the last / second-to-last dimension, diagonal paving,
+ * dense output -- the paper's H and V with any parameters) runs a kernel specialised for its
+ * parameters at run time: compiled with NVRTC on the first call for that filter and array shape
+ * (a fraction of a second, host side), cached for the process.  Without NVRTC, and for every other
+ * filter, a statically compiled generic kernel runs.  Results are identical either way. */
 AOL_API aol_status_t aol_filter_apply(const aol_filter_t* f, const int32_t* d_in, int32_t* d_out, cudaStream_t s);
 
 /* Two repetitions chained -- f2 consumes f1's output array -- in ONE kernel: d_out = f2(f1(d_in)), the
@@ -333,7 +338,9 @@ AOL_API aol_status_t aol_filter_apply(const aol_filter_t* f, const int32_t* d_in
  * each dimension (the paper's H and V output tilers are), f2's output tiler does not wrap, ranks <= 4 and
  * patterns <= 16 elements; otherwise the two filters run as two launches through d_workspace (>= the
  * intermediate array's bytes; NULL -> AOL_E_WORKSPACE naming the reason).  f1.out.array_shape must equal
- * f2.in.array_shape.  d_in / d_out int32 shaped f1.in / f2.out arrays, 4-byte aligned.  Async on s. */
+ * f2.in.array_shape.  d_in / d_out int32 shaped f1.in / f2.out arrays, 4-byte aligned.  Async on s.
+ * A row filter followed by a column filter (the paper's H -> V shape, any parameters) runs a kernel
+ * specialised at run time as for aol_filter_apply (first call per filter pair and shape compiles). */
 AOL_API aol_status_t aol_filter_chain_apply(const aol_filter_t* f1, const aol_filter_t* f2, const int32_t* d_in,
                                             int32_t* d_out, void* d_workspace, size_t ws_bytes, cudaStream_t s);
 
