@@ -295,9 +295,14 @@ def host_cpu():
 # seeded generator synth/ (its C/OpenMP form, untimed); only the oracle calls are timed.
 
 def oracle_threads():
+    """Host threads for the oracle: every core, capped by OpenMP's limit -- except under torch.distributed.run
+    (which sets OMP_NUM_THREADS=1 per rank), where rank 0 alone runs the records' oracle checks while the other
+    ranks wait, so it takes every core."""
     import oracle
 
     cores = os.cpu_count() or 1
+    if int(os.environ.get("WORLD_SIZE", "1")) > 1:
+        return cores
     mt = oracle.max_threads()
     return max(1, min(cores, mt if mt > 0 else cores))
 
