@@ -388,7 +388,7 @@ aol_status_t frame_ex(const void* d_in, aol_dtype_t in_dtype, void* d_out, aol_d
     if (st != AOL_OK) return st;
     if (frames == 0) return AOL_OK;
     FusedPlan plan;
-    st = plan_fused(in_dtype, out_dtype, d_in, d_out, frames, channels, H, W, opts, &plan);
+    st = plan_fused(in_dtype, out_dtype, d_in, d_out, frames, channels, H, W, opts, &plan, d_cs != nullptr);
     if (st != AOL_OK) return st;
     return launch_fused(plan, d_in, in_dtype, d_out, frames, channels, H, W, d_cs, s);
 }

@@ -81,7 +81,7 @@ void fill_plan_info(const FusedPlan& p, aol_plan_t* out);
 
 aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void* d_in, const void* d_out,
                         int64_t frames, int64_t channels, int64_t H, int64_t W, const aol_launch_opts_t* opts,
-                        FusedPlan* plan);
+                        FusedPlan* plan, bool checksum = true);
 aol_status_t launch_fused(const FusedPlan& plan, const void* d_in, aol_dtype_t in_dtype, void* d_out,
                           int64_t frames, int64_t channels, int64_t H, int64_t W, uint64_t* d_cs, cudaStream_t s);
 

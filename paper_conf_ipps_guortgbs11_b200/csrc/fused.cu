@@ -201,7 +201,7 @@ aol_status_t launch_generic(const FusedPlan& plan, const void* d_in, void* d_out
 
 aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void* d_in, const void* d_out,
                         int64_t frames, int64_t channels, int64_t H, int64_t W, const aol_launch_opts_t* opts,
-                        FusedPlan* plan) {
+                        FusedPlan* plan, bool checksum) {
     DeviceInfo dev;
     aol_status_t st = device_info(&dev);
     if (st != AOL_OK) return st;
@@ -259,6 +259,11 @@ aol_status_t plan_fused(aol_dtype_t in_dtype, aol_dtype_t out_dtype, const void*
                                     : rows_per_stage(in_dtype, W, o.flags) == 1 ? 0 : int(geom.stage_stride) / 2;
                 const int target = (kInflightBytesPerSM / cps + half) / int(geom.stage_stride);
                 stages = std::min(stages, std::max(2, target));
+                // planar 8-bit samples with int32 outputs and no checksum epilogue: the lighter consumer runs
+                // ahead of the memory side and a ring of half that depth keeps DRAM efficiency (HD 0.567 -> 0.488
+                // ms at 6 stages instead of 11; with the epilogue 11 stays best, 0.478;
+                // profiles/r02_nocs_stage_sweep.jsonl)
+                if (!checksum && in_dtype == AOL_U8 && out_es == 4) stages = std::min(stages, std::max(2, (target + 1) / 2));
             }
             int occ = 0;
             const int smem = smem_bytes(geom, stages);
