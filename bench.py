@@ -725,6 +725,11 @@ def record_f1(aol, peak, a, frame0, F, d2_cs):
         for odt, oname in ((torch.int32, "int32"), (torch.int16, "int16")):
             z = torch.empty((F, C, Ho, Wo), dtype=odt, device="cuda")
             cs = torch.empty(F, dtype=torch.uint64, device="cuda")
+            # the 8-bit kernels draw enough power that back-to-back variants run into the board's power cap
+            # (sw_power_cap); a second idle before each one measures it as a separate `bench.py --dtype ...` run
+            # would (the clocks sampled during the timing are reported either way)
+            torch.cuda.synchronize()
+            time.sleep(1.0)
             with ClockSampler(torch.cuda.current_device()) as clk:
                 med, mn = timed(lambda: fn(xin, out=z, checksums=cs), inner=5)
                 # the headline's method as well: 50 calls back to back between one event pair
